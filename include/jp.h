@@ -1,0 +1,249 @@
+/*
+ * include/jp.h -- C ABI of libjp.so, the B200 (sm_100a) loop-mode engine after
+ * Japonica (Han, Zhang, Lam, Wang, ICPP'13).  Citations "P:L<n>" point at
+ * /root/reference/PAPER.md lines; "reading Ax" points at DESIGN.md Sec.3.
+ *
+ * What the library does (P:L17-43 abstract; P:L359-380 and Fig. 2):
+ * it executes the iteration space of one annotated loop on the GPU in one of
+ * three modes chosen from a profiled dependency density --
+ *   DOALL  no cross-iteration dependence,
+ *   PRIVATIZED  (private(list) P:L276) only false
+ *               (WAR/WAW) dependences, last-writer-wins write-back,
+ *   GPU-TLS     (mode B P:L367-375) windowed speculative execution,
+ *               RAW check, in-order commit up to the first violator, restart.
+ *
+ * Conventions (all functions):
+ *  - Every pointer is a DEVICE pointer on the current CUDA device unless its
+ *    comment says (host).  The caller owns every buffer, including workspace;
+ *    the library never allocates device memory and keeps no per-loop state.
+ *  - Functions are stream-ordered on `st` and return after enqueueing, EXCEPT
+ *    those documented "syncs": they synchronize `st` before returning because
+ *    they fill a host struct or must decide a status from device data.
+ *  - Errors never abort.  JP_ERR_INDEX (reading A13: an index outside its
+ *    array) is detected before any array is modified.  jp_last_error() gives a
+ *    thread-local message for the last non-OK status.
+ *  - There is no CPU fallback: without a CUDA device every compute entry point
+ *    returns JP_ERR_CUDA.
+ */
+#ifndef JP_H
+#define JP_H
+#include <stddef.h>
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+typedef struct CUstream_st *jp_stream_t;   /* == cudaStream_t; NULL = legacy default stream */
+
+typedef enum { JP_OK = 0, JP_ERR_ARG = -1, JP_ERR_CUDA = -2, JP_ERR_WORKSPACE = -3,
+               JP_ERR_ILLEGAL_MODE = -4, JP_ERR_INDEX = -5, JP_ERR_UNSUPPORTED = -6 } jp_status;
+typedef enum { JP_I32 = 0, JP_F32 = 1 } jp_dtype;
+/* The fixed set of templated loop-body opcodes (BASELINE.json north_star).
+ * Reads precede writes unless marked "covered".  int32 wraps (reading A11);
+ * fp32 is one IEEE RN-even op per operator, never contracted (reading A12).
+ *   JP_OP_ADD_C    A[w[i]] = A[r[i]] + c0
+ *   JP_OP_SAXPY    Y[w[i]] = c0*X[r[i]] + Y[w[i]]                 (Y in slot A)
+ *   JP_OP_PRIV_TMP T[s[i]] = c0*X[r[i]]; Y[w[i]] = T[s[i]] + c1   (T covered; Y in slot A)
+ *   JP_OP_STENCIL2 A[w[i]] = (A[r[i]] + A[r2[i]]) * c0           (Gauss-Seidel shape) */
+typedef enum { JP_OP_ADD_C = 0, JP_OP_SAXPY = 1, JP_OP_PRIV_TMP = 2, JP_OP_STENCIL2 = 3 } jp_op;
+/* Fig. 2(b): A/D' -> DOALL, D -> PRIVATIZED, B -> TLS, C -> SEQ_RECOMMENDED
+ * (mode C is "dispatch to CPU"; there is no CPU path, so it is flagged and executed as TLS). */
+typedef enum { JP_MODE_DOALL = 0, JP_MODE_PRIVATIZED = 1, JP_MODE_TLS = 2,
+               JP_MODE_SEQ_RECOMMENDED = 3 } jp_mode;
+/* scheme(s) clause, Table I: sharing (default) or stealing (Sec. V). */
+typedef enum { JP_SCHED_SHARING = 0, JP_SCHED_STEALING = 1 } jp_scheme;
+
+typedef union { int32_t i; float f; } jp_scalar;
+
+/* Loop descriptor.  Index arrays are int32 [n]; NULL means identity (index i).
+ * Element arrays are 4-byte int32 or fp32 per `dtype`; A, X, T must not alias
+ * each other (reading A14).  Global iteration id of local iteration i is
+ * iter_base + i (used by stamps and keys so that chunks/ranks compose); all
+ * global ids must be < 2^31 - 1.                                               */
+typedef struct {
+  int64_t n;                    /* trip count, 0 <= n, iter_base + n <= 2^31-2        */
+  int64_t iter_base;            /* global id of local iteration 0                     */
+  int32_t op;                   /* jp_op                                              */
+  int32_t dtype;                /* jp_dtype                                           */
+  const int32_t *r, *r2, *w, *s;
+  void *A; int64_t len_A;       /* ADD_C/STENCIL2: A;  SAXPY/PRIV_TMP: Y (in/out)     */
+  const void *X; int64_t len_X; /* read-only operand (SAXPY, PRIV_TMP)                */
+  void *T; int64_t len_T;       /* private(list) scratch, live-out (PRIV_TMP)         */
+  jp_scalar c0, c1;
+} jp_loop;
+
+/* Dependency density (reading A1; model cited from ref [4]):
+ * iteration fractions over the whole loop, any distance, element granularity.
+ *   raw_i: an exposed read of i was written by some earlier iteration
+ *   war_i: a write of i hits an address read (exposed or covered) earlier
+ *   waw_i: a write of i hits an address written earlier                     */
+typedef struct {
+  int64_t n, raw_iters, war_iters, waw_iters;
+  int64_t first_raw_iter;       /* global id, -1 if none                              */
+  double d_raw, d_war, d_waw;   /* *_iters / n  (0 when n == 0)                        */
+} jp_profile;
+
+typedef struct { int64_t committed, executed, windows, violations; } jp_tls_stats;
+
+/* TLS window policy (reading A8).  window > 0: fixed W.  window == 0: adaptive,
+ * W0 = clamp(pow2ceil(ceil(4n/raw)),32,w_max) with a profile (w_max if raw == 0,
+ * 4096 without profile), then W <- clamp(pow2ceil(2*max(c,16)), 32, w_max)
+ * after a window that committed c iterations.  path: 0 auto, 1 single-CTA
+ * shared-memory path (W <= 4096), 2 cooperative all-SM path (HBM stamps).     */
+typedef struct { int64_t window; int64_t w_max; int32_t path; int32_t reserved; } jp_tls_cfg;
+
+typedef struct {
+  int32_t scheme;               /* jp_scheme                                          */
+  int32_t tls_path;             /* jp_tls_cfg.path                                    */
+  double tau_high;              /* Fig. 2(b) "(Density > N)" threshold, reading A4 (0.25) */
+  int64_t chunk_iters;          /* task size for stealing / sharing (reading A17)     */
+  int64_t tls_window;           /* jp_tls_cfg.window                                  */
+  int64_t tls_w_max;            /* jp_tls_cfg.w_max                                   */
+} jp_sched_cfg;
+
+typedef struct {
+  int32_t mode;                 /* jp_mode of the loop (STEALING: of the first task)  */
+  int32_t profiled;             /* 0 when decided statically (all indices NULL)       */
+  jp_profile prof;
+  jp_tls_stats tls;
+  int64_t n_tasks;              /* STEALING: same-mode chunk runs                     */
+  int64_t n_batches;            /* STEALING: topological batches                      */
+  int64_t task_mode_iters[4];   /* iterations executed per jp_mode                    */
+} jp_sched_result;
+
+/* ---- workspace -------------------------------------------------------------
+ * One caller-owned device buffer (256-byte aligned base).  Its regions have
+ * FIXED offsets that depend only on the loop (op, which index arrays are NULL,
+ * lengths, n), in the order header, profile tables, keys, TLS tables,
+ * scheduler scratch; jp_workspace_bytes(L, uses) is the end of the furthest
+ * region any of the requested uses (JP_WS_* bits) needs, so a buffer sized for
+ * more uses serves every smaller one.  Functions return JP_ERR_WORKSPACE when
+ * ws_bytes is too small for what they touch.                                   */
+enum { JP_WS_PROFILE = 1, JP_WS_PRIV = 2, JP_WS_TLS = 4, JP_WS_SCHED = 8, JP_WS_ALL = 15 };
+size_t jp_workspace_bytes(const jp_loop *L /* host */, int32_t uses);
+/* region ids: 0 header, 1 minW(A) int32, 2 minR(A) int32, 3 minW(T), 4 minR(T),
+ * 5 keys(A) int64, 6 keys(T) int64, 7 tls stamps(A) u64, 8 tls commit(A) u64,
+ * 9 (reserved), 10 tls commit(T) u64, 11 scheduler scratch.  Stamp tables hold
+ * INT32_MAX - gid (empty = -1) so that an all_reduce MAX over int32 yields the
+ * global first writer/reader; keys hold (gid+1)<<32 | bits32(value) (empty = 0)
+ * so that an all_reduce MAX over int64 yields the global last writer.  bytes = 0
+ * when the loop does not need the region.  JP_ERR_ARG on a bad id.            */
+jp_status jp_ws_region(const jp_loop *L /* host */, int32_t region, size_t *offset /* host */,
+                       size_t *bytes /* host */);
+
+/* ---- validation (reading A13) ----------------------------------------------
+ * Counts index entries outside their array.  syncs.                          */
+jp_status jp_validate(const jp_loop *L, void *ws, size_t ws_bytes, int64_t *bad /* host */,
+                      jp_stream_t st);
+
+/* ---- profiler (Fig. 1 "Profiler / DD analysis, intra-warp / inter-warp",
+ * P:L127-136) ---------------------------------------------
+ * jp_profile_density = jp_profile_stamp + jp_profile_classify.
+ * stamp:    clears and fills the first-writer / first-reader tables (regions 1-4)
+ *           and validates indices (fused).  Does not sync.
+ * classify: per iteration raw/war/waw flags against the tables, counts, optional
+ *           raw_bits (uint32[ceil(n/32)], bit i%32 of word i/32 = raw_i) and
+ *           optional chunk_counts (int64 [ceil(n/chunk_iters)][3] = raw,war,waw
+ *           per chunk of local iterations; chunk_iters % 32 == 0; zeroed by the
+ *           call).  syncs; returns JP_ERR_INDEX (nothing modified) if the stamp
+ *           pass saw a bad index.                                              */
+jp_status jp_profile_stamp(const jp_loop *L, void *ws, size_t ws_bytes, jp_stream_t st);
+jp_status jp_profile_classify(const jp_loop *L, void *ws, size_t ws_bytes, uint32_t *raw_bits,
+                              int64_t chunk_iters, int64_t *chunk_counts,
+                              jp_profile *out /* host */, jp_stream_t st);
+jp_status jp_profile_density(const jp_loop *L, void *ws, size_t ws_bytes, uint32_t *raw_bits,
+                             int64_t chunk_iters, int64_t *chunk_counts,
+                             jp_profile *out /* host */, jp_stream_t st);
+
+/* Fig. 2(b) decision (host only): all index arrays NULL -> DOALL ("determined
+ * DOALL"); d_raw > tau_high -> SEQ_RECOMMENDED (mode C); d_raw > 0
+ * -> TLS (mode B); d_war > 0 or d_waw > 0 -> PRIVATIZED (mode D); else DOALL
+ * (D').  p may be NULL only for the all-NULL case (else JP_ERR_ARG -> -1).   */
+int32_t jp_select_mode(const jp_loop *L /* host */, const jp_profile *p /* host, nullable */,
+                       double tau_high);
+
+/* ---- DOALL -------------------------------------------------------
+ * Executes all n iterations in place with no protection.  With a profile (host,
+ * nullable) that shows any dependence: JP_ERR_ILLEGAL_MODE.  Without a profile
+ * the caller asserts legality.  If index arrays are present and p == NULL the
+ * indices are validated first (syncs).                                        */
+jp_status jp_run_doall(const jp_loop *L, const jp_profile *p, void *ws, size_t ws_bytes,
+                       jp_stream_t st);
+
+/* ---- PRIVATIZED, PE(V) (readings A9, A10) -------------
+ * Exposed reads see the pre-loop values; covered reads see the iteration's own
+ * private copy; every array that some iteration reaches through a non-identity
+ * index is written through packed last-writer keys and updated after all
+ * iterations; identity-only arrays are stored directly.
+ * With a profile showing d_raw > 0: JP_ERR_ILLEGAL_MODE.  Validation as DOALL.
+ * Split form for multi-GPU: jp_priv_stream fills the key regions (5, 6; zeroed
+ * by the call when `clear_keys`), the caller may all_reduce MAX them, then
+ * jp_priv_finalize applies them.                                              */
+jp_status jp_run_privatized(const jp_loop *L, const jp_profile *p, void *ws, size_t ws_bytes,
+                            jp_stream_t st);
+jp_status jp_priv_stream(const jp_loop *L, const jp_profile *p, void *ws, size_t ws_bytes,
+                         int32_t clear_keys, jp_stream_t st);
+jp_status jp_priv_finalize(const jp_loop *L, void *ws, size_t ws_bytes, jp_stream_t st);
+
+/* ---- GPU-TLS (mode B P:L367-375; readings A6, A7, A8) -------------
+ * Windows [ws, we): speculative execution into per-iteration write logs
+ * (shadow buffers) with read addresses kept as metadata
+ * (P:L326-330); RAW check of every exposed read against earlier in-window
+ * writers; commit of the prefix [ws, fv) up to the first violator fv with
+ * last-writer-wins; restart at fv.  Always legal.  The whole
+ * window loop runs inside one persistent kernel.  stats (host, nullable): if
+ * non-NULL the call syncs.  prof (host, nullable) feeds the adaptive policy and
+ * lets the commit skip WAW resolution when waw_iters == 0.                   */
+jp_status jp_run_tls(const jp_loop *L, const jp_tls_cfg *cfg /* host */, const jp_profile *prof,
+                     void *ws, size_t ws_bytes, jp_tls_stats *stats, jp_stream_t st);
+
+/* ---- scheduler (Sec. V) -----------------------------------------------
+ * One GPU, whole loop: static DOALL check, profile, Fig. 2(b) mode, run.
+ * scheme STEALING: per-chunk profile; maximal same-mode chunk runs become
+ * tasks (Alg. 1 P:L426-437 job pool); tasks that touch a common address with a
+ * write are ordered (PDG reading A19), conflict-free tasks of one topological
+ * batch run concurrently on separate streams (the TLS task on one SM, the
+ * partitioned tasks on the rest).  syncs.                                     */
+jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfg /* host */, void *ws,
+                      size_t ws_bytes, jp_sched_result *res /* host */, jp_stream_t st);
+/* Same, with every array pointer of L_host on the HOST (pinned for speed): the
+ * arrays are copied into `stage` (device, >= jp_stage_bytes), scheduled, and
+ * the written arrays copied back.  syncs.                                      */
+size_t jp_stage_bytes(const jp_loop *L_host /* host */);
+jp_status jp_schedule_host(const jp_loop *L_host /* host */, const jp_sched_cfg *cfg,
+                           void *stage, size_t stage_bytes, void *ws, size_t ws_bytes,
+                           jp_sched_result *res /* host */, jp_stream_t st);
+
+/* ---- multi-GPU plan (host only; P:L342-358 task sharing, P:L426-460 stealing) ----
+ * Task sharing: boundary formula Cg*Fg/(Cg*Fg + Cc*Fc) (garbled at
+ * L355; reading A15) generalised to `world` devices with weights[k] = C_k*F_k:
+ * rank k gets [floor(n*S_k), floor(n*S_{k+1})) with S_k the prefix sum of the
+ * normalised weights (S_world = 1 -> n).  weights NULL = equal.
+ * ranges: (host) int64 [world][2].                                            */
+jp_status jp_plan_sharing(int64_t n, int32_t world, const double *weights /* host */,
+                          int64_t *ranges /* host */);
+/* Task stealing (Alg. 1, readings A16, A18) as a deterministic discrete-event
+ * plan: tasks (host int64 [n_tasks][3] = start, end, mode) are cut into chunks
+ * of chunk_iters (TLS tasks stay whole and pinned to rank 0), dealt to per-rank
+ * deques by task sharing, executed head-first at speed[k] iterations per unit
+ * time (speed_tls for TLS), and an idle rank steals from the TAIL of the deque
+ * with the most remaining iterations (ties: lowest rank).  Output (host):
+ * owner[c] for each chunk in order, and n_chunks via *n_out (must be <= cap).  */
+jp_status jp_plan_stealing(const int64_t *tasks, int64_t n_tasks, int32_t world,
+                           int64_t chunk_iters, const double *speed, double speed_tls,
+                           int64_t *chunks /* host [cap][4]: start,end,mode,owner */,
+                           int64_t cap, int64_t *n_out, int64_t *stolen_out);
+
+/* Apply packed last-writer keys: arr[a] = keys[a] ? lo32(keys[a]) : arr[a]. */
+jp_status jp_merge_apply(void *arr, int64_t len, const int64_t *keys, jp_stream_t st);
+
+const char *jp_last_error(void);
+const char *jp_version(void);
+/* Number of kernels this library has launched in this process (for bench.py). */
+int64_t jp_launch_count(void);
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* JP_H */

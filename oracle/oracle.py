@@ -109,6 +109,11 @@ def run_seq(loop: Loop):
     return st, L.A, L.T
 
 
+def run_seq_inplace(loop: Loop) -> int:
+    """Sequential definition on the loop's own arrays (no copy; used for timing)."""
+    return _load().jpo_run_seq(C.byref(loop._c()))
+
+
 def run_order(loop: Loop, perm):
     L = loop.copy()
     perm = np.ascontiguousarray(perm, dtype=np.int64)

@@ -1,0 +1,261 @@
+"""jp-b200: the Japonica (ICPP'13) loop-mode hot path on B200 (sm_100a).
+
+A thin binding over ``libjp.so`` (C ABI declared in ``include/jp.h``).  Functions
+keep the C names; this module only turns torch tensors into device pointers,
+the current torch stream into a ``cudaStream_t`` and status codes into
+exceptions.  PyTorch is used for device memory, streams and (in ``dist``)
+process groups -- every step of the loop runs in the CUDA kernels.
+"""
+from __future__ import annotations
+
+import ctypes as C
+
+import torch
+
+from . import _abi
+from ._abi import (  # noqa: F401
+    JP_I32, JP_F32, JP_OP_ADD_C, JP_OP_SAXPY, JP_OP_PRIV_TMP, JP_OP_STENCIL2,
+    JP_MODE_DOALL, JP_MODE_PRIVATIZED, JP_MODE_TLS, JP_MODE_SEQ_RECOMMENDED, MODE_NAMES,
+    JP_SCHED_SHARING, JP_SCHED_STEALING, JP_WS_PROFILE, JP_WS_PRIV, JP_WS_TLS, JP_WS_SCHED, JP_WS_ALL,
+    REGIONS, JPError, check, lib,
+)
+
+__all__ = [
+    "Loop", "workspace", "jp_workspace_bytes", "jp_ws_region", "jp_validate", "jp_profile_stamp",
+    "jp_profile_classify", "jp_profile_density", "jp_select_mode", "jp_run_doall", "jp_run_privatized",
+    "jp_priv_stream", "jp_priv_finalize", "jp_run_tls", "jp_schedule", "jp_stage_bytes", "jp_schedule_host",
+    "jp_plan_sharing", "jp_plan_stealing", "jp_merge_apply", "jp_last_error", "jp_version", "jp_launch_count",
+]
+
+_EL = {JP_I32: torch.int32, JP_F32: torch.float32}
+
+
+def _ptr(t):
+    return None if t is None else t.data_ptr()
+
+
+def _stream(stream=None):
+    if stream is not None:
+        return stream.cuda_stream if hasattr(stream, "cuda_stream") else int(stream)
+    if torch.cuda.is_available():
+        return torch.cuda.current_stream().cuda_stream
+    return None
+
+
+class Loop:
+    """A loop descriptor over torch tensors (device, or pinned host for jp_schedule_host).
+
+    op/dtype as in jp.h; index tensors are int32 [n] or None (identity);
+    A (or Y), X, T are int32/float32 1-D tensors.  The tensors are referenced,
+    not copied: the kernels update A (and T) in place."""
+
+    def __init__(self, op, dtype, n, A, r=None, r2=None, w=None, s=None, X=None, T=None, c0=0, c1=0,
+                 iter_base=0):
+        el = _EL[dtype]
+        for name, t in (("A", A), ("X", X), ("T", T)):
+            if t is not None and (t.dtype != el or not t.is_contiguous()):
+                raise ValueError(f"{name} must be a contiguous {el} tensor")
+        for name, t in (("r", r), ("r2", r2), ("w", w), ("s", s)):
+            if t is not None and (t.dtype != torch.int32 or not t.is_contiguous() or t.numel() < n):
+                raise ValueError(f"{name} must be a contiguous int32 tensor of >= n entries")
+        self.tensors = dict(A=A, r=r, r2=r2, w=w, s=s, X=X, T=T)
+        self.op, self.dtype, self.n = int(op), int(dtype), int(n)
+        c = _abi.jp_loop()
+        c.n, c.iter_base, c.op, c.dtype = self.n, int(iter_base), self.op, self.dtype
+        c.r, c.r2, c.w, c.s = _ptr(r), _ptr(r2), _ptr(w), _ptr(s)
+        c.A, c.len_A = _ptr(A), (0 if A is None else A.numel())
+        c.X, c.len_X = _ptr(X), (0 if X is None else X.numel())
+        c.T, c.len_T = _ptr(T), (0 if T is None else T.numel())
+        for slot, v in (("c0", c0), ("c1", c1)):
+            sc = _abi.jp_scalar()
+            if dtype == JP_F32:
+                sc.f = float(v)
+            else:
+                sc.i = int(v) - (1 << 32) if int(v) >= (1 << 31) else int(v)
+            setattr(c, slot, sc)
+        self.c = c
+
+    @classmethod
+    def from_workload(cls, wl, iter_base: int = 0):
+        return cls(wl.op, wl.dtype, wl.n, wl.A, r=wl.r, r2=wl.r2, w=wl.w, s=wl.s, X=wl.X, T=wl.T, c0=wl.c0,
+                   c1=wl.c1, iter_base=iter_base)
+
+    @property
+    def ref(self):
+        return C.byref(self.c)
+
+
+def _prof_dict(p: _abi.jp_profile) -> dict:
+    return {k: getattr(p, k) for k, _ in _abi.jp_profile._fields_}
+
+
+def _prof_struct(p) -> _abi.jp_profile | None:
+    if p is None:
+        return None
+    if isinstance(p, _abi.jp_profile):
+        return p
+    s = _abi.jp_profile()
+    for k, _ in _abi.jp_profile._fields_:
+        setattr(s, k, p[k])
+    return s
+
+
+def _pref(p):
+    s = _prof_struct(p)
+    return None if s is None else C.byref(s)
+
+
+def jp_workspace_bytes(loop: Loop, uses: int = JP_WS_ALL) -> int:
+    return int(lib().jp_workspace_bytes(loop.ref, uses))
+
+
+def workspace(loop: Loop, uses: int = JP_WS_ALL, device="cuda") -> torch.Tensor:
+    """A caller-owned device workspace (torch allocations are >= 256-byte aligned)."""
+    return torch.empty(max(jp_workspace_bytes(loop, uses), 256), dtype=torch.uint8, device=device)
+
+
+def _ws(ws):
+    return (None, 0) if ws is None else (ws.data_ptr(), ws.numel())
+
+
+def jp_ws_region(loop: Loop, region) -> tuple[int, int]:
+    rid = REGIONS[region] if isinstance(region, str) else int(region)
+    off, nb = C.c_size_t(), C.c_size_t()
+    check(lib().jp_ws_region(loop.ref, rid, C.byref(off), C.byref(nb)))
+    return off.value, nb.value
+
+
+def jp_validate(loop: Loop, ws, stream=None) -> int:
+    bad = C.c_int64()
+    p, nb = _ws(ws)
+    st = lib().jp_validate(loop.ref, p, nb, C.byref(bad), _stream(stream))
+    if st not in (_abi.JP_OK, _abi.JP_ERR_INDEX):
+        check(st)
+    return bad.value
+
+
+def jp_profile_stamp(loop: Loop, ws, stream=None):
+    p, nb = _ws(ws)
+    check(lib().jp_profile_stamp(loop.ref, p, nb, _stream(stream)))
+
+
+def jp_profile_classify(loop: Loop, ws, raw_bits=None, chunk_iters=0, chunk_counts=None, stream=None) -> dict:
+    out = _abi.jp_profile()
+    p, nb = _ws(ws)
+    check(lib().jp_profile_classify(loop.ref, p, nb, _ptr(raw_bits), int(chunk_iters), _ptr(chunk_counts),
+                                    C.byref(out), _stream(stream)))
+    return _prof_dict(out)
+
+
+def jp_profile_density(loop: Loop, ws, raw_bits=None, chunk_iters=0, chunk_counts=None, stream=None) -> dict:
+    out = _abi.jp_profile()
+    p, nb = _ws(ws)
+    check(lib().jp_profile_density(loop.ref, p, nb, _ptr(raw_bits), int(chunk_iters), _ptr(chunk_counts),
+                                   C.byref(out), _stream(stream)))
+    return _prof_dict(out)
+
+
+def jp_select_mode(loop: Loop, prof=None, tau_high: float = 0.25) -> int:
+    m = lib().jp_select_mode(loop.ref, _pref(prof), float(tau_high))
+    if m < 0:
+        raise JPError(_abi.JP_ERR_ARG, lib().jp_last_error().decode())
+    return m
+
+
+def jp_run_doall(loop: Loop, prof=None, ws=None, stream=None):
+    p, nb = _ws(ws)
+    check(lib().jp_run_doall(loop.ref, _pref(prof), p, nb, _stream(stream)))
+
+
+def jp_run_privatized(loop: Loop, prof=None, ws=None, stream=None):
+    p, nb = _ws(ws)
+    check(lib().jp_run_privatized(loop.ref, _pref(prof), p, nb, _stream(stream)))
+
+
+def jp_priv_stream(loop: Loop, prof=None, ws=None, clear_keys=True, stream=None):
+    p, nb = _ws(ws)
+    check(lib().jp_priv_stream(loop.ref, _pref(prof), p, nb, int(bool(clear_keys)), _stream(stream)))
+
+
+def jp_priv_finalize(loop: Loop, ws, stream=None):
+    p, nb = _ws(ws)
+    check(lib().jp_priv_finalize(loop.ref, p, nb, _stream(stream)))
+
+
+def jp_run_tls(loop: Loop, window=0, w_max=65536, path=0, prof=None, ws=None, stats=True, stream=None):
+    cfg = _abi.jp_tls_cfg(int(window), int(w_max), int(path), 0)
+    st = _abi.jp_tls_stats()
+    p, nb = _ws(ws)
+    check(lib().jp_run_tls(loop.ref, C.byref(cfg), _pref(prof), p, nb, C.byref(st) if stats else None,
+                           _stream(stream)))
+    return {k: getattr(st, k) for k, _ in _abi.jp_tls_stats._fields_} if stats else None
+
+
+def sched_cfg(scheme=JP_SCHED_SHARING, tau_high=0.25, chunk_iters=65536, tls_window=0, tls_w_max=4096,
+              tls_path=0) -> _abi.jp_sched_cfg:
+    return _abi.jp_sched_cfg(int(scheme), int(tls_path), float(tau_high), int(chunk_iters), int(tls_window),
+                             int(tls_w_max))
+
+
+def _res_dict(r: _abi.jp_sched_result) -> dict:
+    return {"mode": r.mode, "mode_name": MODE_NAMES.get(r.mode, "?"), "profiled": r.profiled,
+            "prof": _prof_dict(r.prof), "tls": {k: getattr(r.tls, k) for k, _ in _abi.jp_tls_stats._fields_},
+            "n_tasks": r.n_tasks, "n_batches": r.n_batches, "task_mode_iters": list(r.task_mode_iters)}
+
+
+def jp_schedule(loop: Loop, ws=None, cfg=None, stream=None, **kw) -> dict:
+    cfg = cfg if cfg is not None else sched_cfg(**kw)
+    res = _abi.jp_sched_result()
+    p, nb = _ws(ws)
+    check(lib().jp_schedule(loop.ref, C.byref(cfg), p, nb, C.byref(res), _stream(stream)))
+    return _res_dict(res)
+
+
+def jp_stage_bytes(loop: Loop) -> int:
+    return int(lib().jp_stage_bytes(loop.ref))
+
+
+def jp_schedule_host(loop: Loop, stage, ws=None, cfg=None, stream=None, **kw) -> dict:
+    """loop's tensors live on the HOST (pinned); stage/ws are device buffers."""
+    cfg = cfg if cfg is not None else sched_cfg(**kw)
+    res = _abi.jp_sched_result()
+    p, nb = _ws(ws)
+    check(lib().jp_schedule_host(loop.ref, C.byref(cfg), stage.data_ptr(), stage.numel(), p, nb, C.byref(res),
+                                 _stream(stream)))
+    return _res_dict(res)
+
+
+def jp_plan_sharing(n: int, world: int, weights=None) -> list[tuple[int, int]]:
+    rg = (C.c_int64 * (2 * world))()
+    wt = None if weights is None else (C.c_double * world)(*[float(x) for x in weights])
+    check(lib().jp_plan_sharing(int(n), int(world), wt, rg))
+    return [(rg[2 * k], rg[2 * k + 1]) for k in range(world)]
+
+
+def jp_plan_stealing(tasks, world: int, chunk_iters: int, speed=None, speed_tls: float = 1.0):
+    """tasks: [(start, end, mode)].  Returns (chunks [(start, end, mode, owner)], n_stolen)."""
+    flat = [int(v) for t in tasks for v in t]
+    tk = (C.c_int64 * max(len(flat), 1))(*flat)
+    cap = sum(max(1, -(-(e - s) // chunk_iters)) for s, e, _ in tasks) + len(tasks) + 1
+    out = (C.c_int64 * (4 * cap))()
+    n_out, stolen = C.c_int64(), C.c_int64()
+    sp = None if speed is None else (C.c_double * world)(*[float(x) for x in speed])
+    check(lib().jp_plan_stealing(tk, len(tasks), int(world), int(chunk_iters), sp, float(speed_tls), out, cap,
+                                 C.byref(n_out), C.byref(stolen)))
+    return [tuple(out[4 * c:4 * c + 4]) for c in range(n_out.value)], stolen.value
+
+
+def jp_merge_apply(arr: torch.Tensor, keys: torch.Tensor, stream=None):
+    check(lib().jp_merge_apply(arr.data_ptr(), arr.numel(), keys.data_ptr(), _stream(stream)))
+
+
+def jp_last_error() -> str:
+    return lib().jp_last_error().decode()
+
+
+def jp_version() -> str:
+    return lib().jp_version().decode()
+
+
+def jp_launch_count() -> int:
+    return int(lib().jp_launch_count())

@@ -1,0 +1,796 @@
+// jp_api.cu -- the extern "C" entry points of libjp.so (include/jp.h).
+// Host logic only: argument checks, workspace layout, the Fig. 2(b) decision,
+// the task-sharing / task-stealing plans and the one-GPU scheduler.  Every
+// step of the loop itself runs in the kernels of jp_*.cu.
+#include <algorithm>
+#include <atomic>
+#include <cmath>
+#include <cstdarg>
+#include <cstdio>
+#include <cstring>
+#include <mutex>
+#include <string>
+#include <vector>
+
+#include "jp_host.h"
+
+namespace jp {
+
+static std::atomic<long long> g_launches{0};
+void note_launch(int k) { g_launches.fetch_add(k, std::memory_order_relaxed); }
+
+static thread_local std::string g_err;
+
+static jp_status fail(jp_status s, const char *fmt, ...) {
+  char buf[512];
+  va_list ap;
+  va_start(ap, fmt);
+  vsnprintf(buf, sizeof buf, fmt, ap);
+  va_end(ap);
+  g_err = buf;
+  return s;
+}
+
+int num_sms() {
+  static int cache[64] = {0};
+  int dev = 0;
+  cudaGetDevice(&dev);
+  if (dev < 0 || dev >= 64) dev = 0;
+  if (!cache[dev]) {
+    int v = 0;
+    cudaDeviceGetAttribute(&v, cudaDevAttrMultiProcessorCount, dev);
+    cache[dev] = v > 0 ? v : 1;
+  }
+  return cache[dev];
+}
+
+cudaError_t launch_check() { return cudaGetLastError(); }
+
+static jp_status cuda_fail(cudaError_t e, const char *where) {
+  return fail(JP_ERR_CUDA, "%s: %s", where, cudaGetErrorString(e));
+}
+
+static bool have_device() {
+  int n = 0;
+  if (cudaGetDeviceCount(&n) != cudaSuccess || n == 0) {
+    cudaGetLastError();
+    return false;
+  }
+  return true;
+}
+
+static size_t al256(size_t x) { return (x + 255) & ~(size_t)255; }
+
+// index arrays the opcode actually uses
+static void used_idx(int op, bool &r, bool &r2, bool &w, bool &s) {
+  r = true; w = true;
+  r2 = op == JP_OP_STENCIL2;
+  s = op == JP_OP_PRIV_TMP;
+}
+
+Job make_job(const jp_loop *L) {
+  Job j;
+  bool ur, ur2, uw, us;
+  used_idx(L->op, ur, ur2, uw, us);
+  j.op = L->op;
+  j.dt = L->dtype;
+  DLoop &d = j.d;
+  d.n = L->n;
+  d.base = L->iter_base;
+  d.ioff = 0;
+  d.r = ur ? L->r : nullptr;
+  d.r2 = ur2 ? L->r2 : nullptr;
+  d.w = uw ? L->w : nullptr;
+  d.s = us ? L->s : nullptr;
+  d.A = static_cast<uint32_t *>(L->A);
+  d.lenA = L->len_A;
+  d.X = static_cast<const uint32_t *>(L->X);
+  d.lenX = L->len_X;
+  d.T = static_cast<uint32_t *>(L->T);
+  d.lenT = L->len_T;
+  d.c0 = (uint32_t)L->c0.i;
+  d.c1 = (uint32_t)L->c1.i;
+  return j;
+}
+
+static bool has_idx(const Job &j) { return j.d.r || j.d.r2 || j.d.w || j.d.s; }
+
+SchedLayout sched_layout(const jp_loop *L) {
+  SchedLayout s{};
+  Job j = make_job(L);
+  const bool aI = a_indirect(j.op, j.d.r, j.d.r2, j.d.w), tI = t_indirect(j.op, j.d.s);
+  const int64_t nck = (L->n + kSchedMinChunk - 1) / kSchedMinChunk + 1;
+  size_t o = 0;
+  s.counts = o; o = al256(o + 24 * (size_t)nck);
+  s.chunk_task = o; o = al256(o + 4 * (size_t)nck);
+  s.wmA = aI ? o : SIZE_MAX; if (aI) o = al256(o + 8 * (size_t)L->len_A);
+  s.rmA = aI && a_has_reads(j.op) ? o : SIZE_MAX; if (s.rmA != SIZE_MAX) o = al256(o + 8 * (size_t)L->len_A);
+  s.wmT = tI ? o : SIZE_MAX; if (tI) o = al256(o + 8 * (size_t)L->len_T);
+  s.rmT = tI ? o : SIZE_MAX; if (tI) o = al256(o + 8 * (size_t)L->len_T);
+  s.conf = o; o = al256(o + 8 * kMaxTasks);
+  s.tstats = o; o = al256(o + 32 * kMaxTasks);
+  s.total = o;
+  return s;
+}
+
+Layout layout(const jp_loop *L) {
+  Layout lo;
+  memset(&lo, 0, sizeof lo);
+  Job j = make_job(L);
+  const bool aI = a_indirect(j.op, j.d.r, j.d.r2, j.d.w), tI = t_indirect(j.op, j.d.s);
+  size_t off = 0;
+  auto add = [&](int r, size_t bytes) {
+    off = al256(off);
+    lo.off[r] = off;
+    lo.bytes[r] = bytes;
+    off += bytes;
+  };
+  add(R_HEADER, kHeaderBytes);
+  add(R_MINW_A, aI ? 4 * (size_t)L->len_A : 0);
+  add(R_MINR_A, aI && a_has_reads(j.op) ? 4 * (size_t)L->len_A : 0);
+  add(R_MINW_T, tI ? 4 * (size_t)L->len_T : 0);
+  add(R_MINR_T, tI ? 4 * (size_t)L->len_T : 0);
+  add(R_KEYS_A, aI ? 8 * (size_t)L->len_A : 0);
+  add(R_KEYS_T, tI ? 8 * (size_t)L->len_T : 0);
+  add(R_TLS_S_A, aI && j.op != JP_OP_PRIV_TMP ? 8 * (size_t)L->len_A : 0);
+  add(R_TLS_C_A, aI ? 8 * (size_t)L->len_A : 0);
+  add(R_TLS_S_T, 0);
+  add(R_TLS_C_T, tI ? 8 * (size_t)L->len_T : 0);
+  add(R_SCHED, sched_layout(L).total);
+  lo.total = al256(off);
+  return lo;
+}
+
+size_t layout_end(const Layout &lo, int uses) {
+  int last = R_HEADER;
+  if (uses & JP_WS_PROFILE) last = R_MINR_T;
+  if (uses & JP_WS_PRIV) last = std::max(last, (int)R_KEYS_T);
+  if (uses & JP_WS_TLS) last = std::max(last, (int)R_TLS_C_T);
+  if (uses & JP_WS_SCHED) last = R_SCHED;
+  return al256(lo.off[last] + lo.bytes[last]);
+}
+
+}  // namespace jp
+
+using namespace jp;
+
+// ---------------------------------------------------------------------------
+// argument checks
+// ---------------------------------------------------------------------------
+static jp_status check_loop(const jp_loop *L) {
+  if (!L) return fail(JP_ERR_ARG, "loop descriptor is NULL");
+  if (L->op < JP_OP_ADD_C || L->op > JP_OP_STENCIL2) return fail(JP_ERR_UNSUPPORTED, "opcode %d is not templated", L->op);
+  if (L->dtype != JP_I32 && L->dtype != JP_F32) return fail(JP_ERR_UNSUPPORTED, "dtype %d is not templated", L->dtype);
+  if (L->n < 0 || L->iter_base < 0 || L->iter_base + L->n > 2147483646LL)
+    return fail(JP_ERR_ARG, "need 0 <= n, 0 <= iter_base, iter_base + n <= 2^31-2 (n=%lld base=%lld)",
+                (long long)L->n, (long long)L->iter_base);
+  const int64_t lmax = 2147483647LL;
+  if (L->len_A < 0 || L->len_X < 0 || L->len_T < 0 || L->len_A > lmax || L->len_X > lmax || L->len_T > lmax)
+    return fail(JP_ERR_ARG, "array lengths must be in [0, 2^31-1]");
+  if (L->n == 0) return JP_OK;
+  if (!L->A) return fail(JP_ERR_ARG, "A/Y is NULL");
+  const bool usesX = L->op == JP_OP_SAXPY || L->op == JP_OP_PRIV_TMP;
+  if (usesX && !L->X) return fail(JP_ERR_ARG, "X is NULL");
+  if (L->op == JP_OP_PRIV_TMP && !L->T) return fail(JP_ERR_ARG, "T is NULL");
+  // identity accesses must stay inside their arrays (reading A13)
+  auto idn = [&](const int32_t *p, int64_t len, const char *what) -> jp_status {
+    if (!p && L->n > len) return fail(JP_ERR_INDEX, "identity index of %s exceeds its length (%lld > %lld)", what,
+                                      (long long)L->n, (long long)len);
+    return JP_OK;
+  };
+  jp_status s = JP_OK;
+  switch (L->op) {
+    case JP_OP_ADD_C: if ((s = idn(L->r, L->len_A, "r"))) return s; if ((s = idn(L->w, L->len_A, "w"))) return s; break;
+    case JP_OP_SAXPY: if ((s = idn(L->r, L->len_X, "r"))) return s; if ((s = idn(L->w, L->len_A, "w"))) return s; break;
+    case JP_OP_PRIV_TMP:
+      if ((s = idn(L->r, L->len_X, "r"))) return s;
+      if ((s = idn(L->s, L->len_T, "s"))) return s;
+      if ((s = idn(L->w, L->len_A, "w"))) return s;
+      break;
+    default:
+      if ((s = idn(L->r, L->len_A, "r"))) return s;
+      if ((s = idn(L->r2, L->len_A, "r2"))) return s;
+      if ((s = idn(L->w, L->len_A, "w"))) return s;
+  }
+  return JP_OK;
+}
+
+static jp_status check_ws(const jp_loop *L, void *ws, size_t ws_bytes, int uses, Layout &lo) {
+  lo = layout(L);
+  const size_t need = layout_end(lo, uses);
+  if (!ws || ws_bytes < need)
+    return fail(JP_ERR_WORKSPACE, "workspace of %zu bytes is smaller than the %zu bytes needed", ws ? ws_bytes : 0,
+                need);
+  if ((uintptr_t)ws & 255) return fail(JP_ERR_WORKSPACE, "workspace must be 256-byte aligned");
+  return JP_OK;
+}
+
+#define JP_TRY(expr)                  \
+  do {                                \
+    jp_status _s = (expr);            \
+    if (_s != JP_OK) return _s;       \
+  } while (0)
+#define JP_CUDA(expr, where)                        \
+  do {                                              \
+    cudaError_t _e = (expr);                        \
+    if (_e != cudaSuccess) return cuda_fail(_e, where); \
+  } while (0)
+
+static jp_status need_device() {
+  if (!have_device()) return fail(JP_ERR_CUDA, "no CUDA device (libjp.so has no CPU fallback)");
+  return JP_OK;
+}
+
+// validate indices on the device, syncs; JP_ERR_INDEX when any is out of range
+static jp_status validate_sync(const Job &j, void *ws, const Layout &lo, cudaStream_t st, int64_t *bad_out) {
+  int64_t *hdr = at<int64_t>(ws, lo, R_HEADER);
+  JP_CUDA(launch_validate(j, hdr, st), "validate");
+  int64_t bad = 0;
+  JP_CUDA(cudaMemcpyAsync(&bad, &hdr[H_BAD], sizeof bad, cudaMemcpyDeviceToHost, st), "validate D2H");
+  JP_CUDA(cudaStreamSynchronize(st), "validate sync");
+  if (bad_out) *bad_out = bad;
+  if (bad) return fail(JP_ERR_INDEX, "%lld index entries are outside their arrays", (long long)bad);
+  return JP_OK;
+}
+
+extern "C" {
+
+const char *jp_last_error(void) { return g_err.c_str(); }
+const char *jp_version(void) { return "jp-b200 0.1 (sm_100a)"; }
+int64_t jp_launch_count(void) { return g_launches.load(); }
+
+size_t jp_workspace_bytes(const jp_loop *L, int32_t uses) {
+  if (!L || check_loop(L) == JP_ERR_ARG) return 0;
+  return layout_end(layout(L), uses);
+}
+
+jp_status jp_ws_region(const jp_loop *L, int32_t region, size_t *offset, size_t *bytes) {
+  JP_TRY(check_loop(L));
+  if (region < 0 || region >= R_COUNT) return fail(JP_ERR_ARG, "bad region id %d", region);
+  Layout lo = layout(L);
+  if (offset) *offset = lo.off[region];
+  if (bytes) *bytes = lo.bytes[region];
+  return JP_OK;
+}
+
+jp_status jp_validate(const jp_loop *L, void *ws, size_t ws_bytes, int64_t *bad, jp_stream_t st) {
+  jp_status s = check_loop(L);
+  if (s == JP_ERR_INDEX) { if (bad) *bad = -1; return s; }
+  JP_TRY(s);
+  JP_TRY(need_device());
+  Layout lo;
+  JP_TRY(check_ws(L, ws, ws_bytes, 0, lo));
+  return validate_sync(make_job(L), ws, lo, (cudaStream_t)st, bad);
+}
+
+jp_status jp_profile_stamp(const jp_loop *L, void *ws, size_t ws_bytes, jp_stream_t st) {
+  JP_TRY(check_loop(L));
+  JP_TRY(need_device());
+  Layout lo;
+  JP_TRY(check_ws(L, ws, ws_bytes, JP_WS_PROFILE, lo));
+  JP_CUDA(launch_prof_stamp(make_job(L), ws, lo, (cudaStream_t)st), "profile stamp");
+  return JP_OK;
+}
+
+static void fill_profile(jp_profile *out, int64_t n, const int64_t *h) {
+  out->n = n;
+  out->raw_iters = h[H_RAW];
+  out->war_iters = h[H_WAR];
+  out->waw_iters = h[H_WAW];
+  out->first_raw_iter = h[H_FIRST_RAW];   // -1 (all ones) when none
+  out->d_raw = n ? (double)out->raw_iters / (double)n : 0.0;
+  out->d_war = n ? (double)out->war_iters / (double)n : 0.0;
+  out->d_waw = n ? (double)out->waw_iters / (double)n : 0.0;
+}
+
+jp_status jp_profile_classify(const jp_loop *L, void *ws, size_t ws_bytes, uint32_t *raw_bits, int64_t chunk_iters,
+                              int64_t *chunk_counts, jp_profile *out, jp_stream_t stp) {
+  JP_TRY(check_loop(L));
+  if (!out) return fail(JP_ERR_ARG, "profile output is NULL");
+  if (chunk_counts && (chunk_iters <= 0 || chunk_iters % 32))
+    return fail(JP_ERR_ARG, "chunk_iters must be a positive multiple of 32");
+  JP_TRY(need_device());
+  Layout lo;
+  JP_TRY(check_ws(L, ws, ws_bytes, JP_WS_PROFILE, lo));
+  cudaStream_t st = (cudaStream_t)stp;
+  JP_CUDA(launch_prof_classify(make_job(L), ws, lo, raw_bits, chunk_iters, chunk_counts, st), "profile classify");
+  int64_t h[8];
+  JP_CUDA(cudaMemcpyAsync(h, at<int64_t>(ws, lo, R_HEADER), sizeof h, cudaMemcpyDeviceToHost, st), "profile D2H");
+  JP_CUDA(cudaStreamSynchronize(st), "profile sync");
+  if (h[H_BAD]) return fail(JP_ERR_INDEX, "%lld index entries are outside their arrays", (long long)h[H_BAD]);
+  fill_profile(out, L->n, h);
+  return JP_OK;
+}
+
+jp_status jp_profile_density(const jp_loop *L, void *ws, size_t ws_bytes, uint32_t *raw_bits, int64_t chunk_iters,
+                             int64_t *chunk_counts, jp_profile *out, jp_stream_t st) {
+  JP_TRY(jp_profile_stamp(L, ws, ws_bytes, st));
+  return jp_profile_classify(L, ws, ws_bytes, raw_bits, chunk_iters, chunk_counts, out, st);
+}
+
+static int32_t select_mode_counts(int64_t n, int64_t raw, int64_t war, int64_t waw, double tau) {
+  const double d_raw = n ? (double)raw / (double)n : 0.0;
+  if (d_raw > tau) return JP_MODE_SEQ_RECOMMENDED;   // mode C
+  if (raw > 0) return JP_MODE_TLS;                    // mode B
+  if (war > 0 || waw > 0) return JP_MODE_PRIVATIZED;  // mode D
+  return JP_MODE_DOALL;                               // mode D'
+}
+
+int32_t jp_select_mode(const jp_loop *L, const jp_profile *p, double tau_high) {
+  if (check_loop(L) == JP_ERR_ARG || check_loop(L) == JP_ERR_UNSUPPORTED) return -1;
+  Job j = make_job(L);
+  if (!has_idx(j)) return JP_MODE_DOALL;   // "determined DOALL" (mode A), no profile needed
+  if (!p) { fail(JP_ERR_ARG, "a profile is required when index arrays are present"); return -1; }
+  return select_mode_counts(p->n, p->raw_iters, p->war_iters, p->waw_iters, tau_high);
+}
+
+jp_status jp_run_doall(const jp_loop *L, const jp_profile *p, void *ws, size_t ws_bytes, jp_stream_t stp) {
+  JP_TRY(check_loop(L));
+  if (p && (p->raw_iters || p->war_iters || p->waw_iters))
+    return fail(JP_ERR_ILLEGAL_MODE, "DOALL needs d_raw = d_war = d_waw = 0 (profile: %lld/%lld/%lld)",
+                (long long)p->raw_iters, (long long)p->war_iters, (long long)p->waw_iters);
+  JP_TRY(need_device());
+  cudaStream_t st = (cudaStream_t)stp;
+  Job j = make_job(L);
+  if (has_idx(j) && !p) {
+    Layout lo;
+    JP_TRY(check_ws(L, ws, ws_bytes, 0, lo));
+    JP_TRY(validate_sync(j, ws, lo, st, nullptr));
+  }
+  JP_CUDA(launch_doall(j, st), "doall");
+  return JP_OK;
+}
+
+jp_status jp_priv_stream(const jp_loop *L, const jp_profile *p, void *ws, size_t ws_bytes, int32_t clear_keys,
+                         jp_stream_t stp) {
+  JP_TRY(check_loop(L));
+  if (p && p->raw_iters)
+    return fail(JP_ERR_ILLEGAL_MODE, "privatization needs d_raw = 0 (profile: %lld RAW iterations)",
+                (long long)p->raw_iters);
+  JP_TRY(need_device());
+  Layout lo;
+  JP_TRY(check_ws(L, ws, ws_bytes, JP_WS_PRIV, lo));
+  cudaStream_t st = (cudaStream_t)stp;
+  Job j = make_job(L);
+  if (has_idx(j) && !p) JP_TRY(validate_sync(j, ws, lo, st, nullptr));
+  JP_CUDA(launch_priv_stream(j, ws, lo, clear_keys != 0, st), "priv stream");
+  return JP_OK;
+}
+
+jp_status jp_priv_finalize(const jp_loop *L, void *ws, size_t ws_bytes, jp_stream_t st) {
+  JP_TRY(check_loop(L));
+  JP_TRY(need_device());
+  Layout lo;
+  JP_TRY(check_ws(L, ws, ws_bytes, JP_WS_PRIV, lo));
+  JP_CUDA(launch_priv_finalize(make_job(L), ws, lo, (cudaStream_t)st), "priv finalize");
+  return JP_OK;
+}
+
+jp_status jp_run_privatized(const jp_loop *L, const jp_profile *p, void *ws, size_t ws_bytes, jp_stream_t st) {
+  JP_TRY(jp_priv_stream(L, p, ws, ws_bytes, 1, st));
+  return jp_priv_finalize(L, ws, ws_bytes, st);
+}
+
+// choose the TLS path and check its limits
+static jp_status tls_plan(const Job &j, const jp_tls_cfg *cfg, const jp_profile *prof, TlsPlan &tp) {
+  tp.window = cfg ? cfg->window : 0;
+  tp.w_max = cfg && cfg->w_max > 0 ? cfg->w_max : 65536;
+  tp.prof_raw = prof ? prof->raw_iters : -1;
+  if (tp.window < 0) return fail(JP_ERR_ARG, "window must be >= 0");
+  if (tp.window == 0 && tp.w_max < 32) return fail(JP_ERR_ARG, "w_max must be >= 32");
+  const bool hA = a_indirect(j.op, j.d.r, j.d.r2, j.d.w), hT = t_indirect(j.op, j.d.s);
+  tp.waw = (hA || hT) && !(prof && prof->waw_iters == 0);
+  const int64_t wcap = tp.window > 0 ? tp.window : tp.w_max;
+  const int64_t cta_max = (j.op == JP_OP_PRIV_TMP && hA && hT) ? kTlsCtaWmax / 2 : kTlsCtaWmax;
+  int path = cfg ? cfg->path : 0;
+  if (path == 0) path = wcap <= cta_max ? 1 : 2;
+  if (path == 1 && wcap > cta_max)
+    return fail(JP_ERR_UNSUPPORTED, "the single-CTA TLS path holds windows up to %lld iterations", (long long)cta_max);
+  if (path != 1 && path != 2) return fail(JP_ERR_ARG, "bad TLS path %d", path);
+  tp.path = path;
+  return JP_OK;
+}
+
+static jp_status run_tls_job(const jp_loop *L, const Job &j, const jp_tls_cfg *cfg, const jp_profile *prof, void *ws,
+                             size_t ws_bytes, jp_tls_stats *stats, cudaStream_t st) {
+  TlsPlan tp;
+  JP_TRY(tls_plan(j, cfg, prof, tp));
+  Layout lo;
+  JP_TRY(check_ws(L, ws, ws_bytes, tp.path == 2 ? JP_WS_TLS : 0, lo));
+  if (has_idx(j) && !prof) JP_TRY(validate_sync(j, ws, lo, st, nullptr));
+  int64_t *hdr = at<int64_t>(ws, lo, R_HEADER);
+  JP_CUDA(launch_tls(j, ws, lo, tp, &hdr[H_TLS_COMMITTED], st), "tls");
+  if (stats) {
+    int64_t h[4];
+    JP_CUDA(cudaMemcpyAsync(h, &hdr[H_TLS_COMMITTED], sizeof h, cudaMemcpyDeviceToHost, st), "tls D2H");
+    JP_CUDA(cudaStreamSynchronize(st), "tls sync");
+    stats->committed = h[0];
+    stats->executed = h[1];
+    stats->windows = h[2];
+    stats->violations = h[3];
+  }
+  return JP_OK;
+}
+
+jp_status jp_run_tls(const jp_loop *L, const jp_tls_cfg *cfg, const jp_profile *prof, void *ws, size_t ws_bytes,
+                     jp_tls_stats *stats, jp_stream_t st) {
+  JP_TRY(check_loop(L));
+  JP_TRY(need_device());
+  return run_tls_job(L, make_job(L), cfg, prof, ws, ws_bytes, stats, (cudaStream_t)st);
+}
+
+jp_status jp_merge_apply(void *arr, int64_t len, const int64_t *keys, jp_stream_t st) {
+  if (len < 0 || (len > 0 && (!arr || !keys))) return fail(JP_ERR_ARG, "bad merge arguments");
+  JP_TRY(need_device());
+  JP_CUDA(launch_merge_apply(arr, len, keys, (cudaStream_t)st), "merge apply");
+  return JP_OK;
+}
+
+// ---------------------------------------------------------------------------
+// plans (host only)
+// ---------------------------------------------------------------------------
+jp_status jp_plan_sharing(int64_t n, int32_t world, const double *weights, int64_t *ranges) {
+  if (n < 0 || world <= 0 || !ranges) return fail(JP_ERR_ARG, "bad sharing-plan arguments");
+  double total = 0.0;
+  for (int k = 0; k < world; k++) {
+    const double w = weights ? weights[k] : 1.0;
+    if (!(w >= 0.0) || std::isinf(w)) return fail(JP_ERR_ARG, "weights must be finite and >= 0");
+    total += w;
+  }
+  if (!(total > 0.0)) return fail(JP_ERR_ARG, "weights sum to zero");
+  double pre = 0.0;
+  for (int k = 0; k < world; k++) {
+    const int64_t b0 = (int64_t)std::floor((double)n * (pre / total));
+    pre += weights ? weights[k] : 1.0;
+    const int64_t b1 = k == world - 1 ? n : (int64_t)std::floor((double)n * (pre / total));
+    ranges[2 * k] = b0;
+    ranges[2 * k + 1] = b1;
+  }
+  return JP_OK;
+}
+
+jp_status jp_plan_stealing(const int64_t *tasks, int64_t n_tasks, int32_t world, int64_t chunk_iters,
+                           const double *speed, double speed_tls, int64_t *chunks, int64_t cap, int64_t *n_out,
+                           int64_t *stolen_out) {
+  if (!tasks || n_tasks < 0 || world <= 0 || chunk_iters <= 0 || !chunks || !n_out || !(speed_tls > 0.0))
+    return fail(JP_ERR_ARG, "bad stealing-plan arguments");
+  for (int k = 0; k < world; k++)
+    if (speed && !(speed[k] > 0.0)) return fail(JP_ERR_ARG, "speeds must be > 0");
+  struct Ch { int64_t s, e, mode, home, owner; };
+  std::vector<Ch> cs;
+  for (int64_t t = 0; t < n_tasks; t++) {
+    const int64_t s = tasks[3 * t], e = tasks[3 * t + 1], m = tasks[3 * t + 2];
+    if (e < s) return fail(JP_ERR_ARG, "task %lld has end < start", (long long)t);
+    const bool tls = m == JP_MODE_TLS || m == JP_MODE_SEQ_RECOMMENDED;
+    if (tls) { cs.push_back({s, e, m, 0, -1}); continue; }
+    for (int64_t c = s; c < e; c += chunk_iters) cs.push_back({c, std::min(e, c + chunk_iters), m, -1, -1});
+  }
+  if ((int64_t)cs.size() > cap) { *n_out = (int64_t)cs.size(); return fail(JP_ERR_ARG, "plan needs %zu chunks", cs.size()); }
+  // deal the partitionable chunks by task sharing (weights = speeds)
+  std::vector<int64_t> part;
+  for (size_t c = 0; c < cs.size(); c++) if (cs[c].home < 0) part.push_back((int64_t)c);
+  std::vector<int64_t> rg(2 * world);
+  jp_plan_sharing((int64_t)part.size(), world, speed, rg.data());
+  std::vector<std::vector<int64_t>> dq(world), pinned(world);
+  for (int k = 0; k < world; k++)
+    for (int64_t q = rg[2 * k]; q < rg[2 * k + 1]; q++) { cs[part[q]].home = k; dq[k].push_back(part[q]); }
+  for (size_t c = 0; c < cs.size(); c++) if (cs[c].home == 0 && (cs[c].mode == JP_MODE_TLS || cs[c].mode == JP_MODE_SEQ_RECOMMENDED)) pinned[0].push_back((int64_t)c);
+  std::vector<size_t> head(world, 0), tail(world), pin_head(world, 0);
+  for (int k = 0; k < world; k++) tail[k] = dq[k].size();
+  std::vector<double> t(world, 0.0);
+  std::vector<bool> done(world, false);
+  int64_t stolen = 0;
+  while (true) {
+    int k = -1;
+    for (int q = 0; q < world; q++) if (!done[q] && (k < 0 || t[q] < t[k])) k = q;
+    if (k < 0) break;
+    int64_t c = -1;
+    double rate = speed ? speed[k] : 1.0;
+    if (pin_head[k] < pinned[k].size()) { c = pinned[k][pin_head[k]++]; rate = speed_tls; }
+    else if (head[k] < tail[k]) c = dq[k][head[k]++];
+    else {
+      // steal from the TAIL of the deque with the most remaining iterations (ties: lowest rank)
+      int v = -1; int64_t best = 0;
+      for (int q = 0; q < world; q++) {
+        if (q == k) continue;
+        int64_t rem = 0;
+        for (size_t x = head[q]; x < tail[q]; x++) rem += cs[dq[q][x]].e - cs[dq[q][x]].s;
+        if (rem > best) { best = rem; v = q; }
+      }
+      if (v < 0) { done[k] = true; continue; }
+      c = dq[v][--tail[v]];
+      stolen++;
+    }
+    cs[c].owner = k;
+    t[k] += (double)(cs[c].e - cs[c].s) / rate;
+  }
+  for (size_t c = 0; c < cs.size(); c++) {
+    chunks[4 * c] = cs[c].s; chunks[4 * c + 1] = cs[c].e; chunks[4 * c + 2] = cs[c].mode; chunks[4 * c + 3] = cs[c].owner;
+  }
+  *n_out = (int64_t)cs.size();
+  if (stolen_out) *stolen_out = stolen;
+  return JP_OK;
+}
+
+// ---------------------------------------------------------------------------
+// scheduler (one GPU)
+// ---------------------------------------------------------------------------
+static jp_sched_cfg default_cfg() {
+  jp_sched_cfg c;
+  memset(&c, 0, sizeof c);
+  c.scheme = JP_SCHED_SHARING;
+  c.tau_high = 0.25;
+  c.chunk_iters = 65536;
+  c.tls_window = 0;
+  c.tls_w_max = 4096;
+  c.tls_path = 0;
+  return c;
+}
+
+static Job sub_job(const Job &j, int64_t s, int64_t e) {
+  Job k = j;
+  DLoop &d = k.d;
+  d.n = e - s;
+  d.base = j.d.base + s;
+  d.ioff = j.d.ioff + s;
+  if (d.r) d.r += s;
+  if (d.r2) d.r2 += s;
+  if (d.w) d.w += s;
+  if (d.s) d.s += s;
+  return k;
+}
+
+static jp_status run_mode(const jp_loop *L, const Job &j, int mode, const jp_profile *prof, const jp_sched_cfg &c,
+                          void *ws, size_t ws_bytes, jp_sched_result *res, cudaStream_t st) {
+  Layout lo = layout(L);
+  if (mode == JP_MODE_DOALL) {
+    JP_CUDA(launch_doall(j, st), "doall");
+  } else if (mode == JP_MODE_PRIVATIZED) {
+    if (ws_bytes < layout_end(lo, JP_WS_PRIV)) return fail(JP_ERR_WORKSPACE, "workspace too small for privatization");
+    JP_CUDA(launch_priv_stream(j, ws, lo, true, st), "priv stream");
+    JP_CUDA(launch_priv_finalize(j, ws, lo, st), "priv finalize");
+  } else {
+    jp_tls_cfg tc{c.tls_window, c.tls_w_max, c.tls_path, 0};
+    JP_TRY(run_tls_job(L, j, &tc, prof, ws, ws_bytes, &res->tls, st));
+  }
+  res->task_mode_iters[mode] += j.d.n;
+  return JP_OK;
+}
+
+namespace {
+struct StreamPool {
+  std::mutex mu;
+  std::vector<cudaStream_t> s[64];
+  cudaStream_t get(int k) {
+    int dev = 0;
+    cudaGetDevice(&dev);
+    std::lock_guard<std::mutex> g(mu);
+    auto &v = s[dev & 63];
+    while ((int)v.size() <= k) {
+      cudaStream_t x;
+      cudaStreamCreateWithFlags(&x, cudaStreamNonBlocking);
+      v.push_back(x);
+    }
+    return v[k];
+  }
+} g_pool;
+}  // namespace
+
+static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sched_cfg &c, void *ws, size_t ws_bytes,
+                                   jp_sched_result *res, cudaStream_t st) {
+  const int64_t chunk = c.chunk_iters;
+  if (chunk < kSchedMinChunk || chunk % 32) return fail(JP_ERR_ARG, "stealing needs chunk_iters >= 1024, multiple of 32");
+  Layout lo;
+  JP_TRY(check_ws(L, ws, ws_bytes, JP_WS_ALL, lo));
+  SchedLayout sl = sched_layout(L);
+  char *sch = static_cast<char *>(ws) + lo.off[R_SCHED];
+  const int64_t nck = (L->n + chunk - 1) / chunk;
+  int64_t *cc = reinterpret_cast<int64_t *>(sch + sl.counts);
+  // 1. profile with per-chunk counts (global stamps, reading A19)
+  JP_CUDA(launch_prof_stamp(j, ws, lo, st), "profile stamp");
+  JP_CUDA(launch_prof_classify(j, ws, lo, nullptr, chunk, cc, st), "profile classify");
+  std::vector<int64_t> hc(3 * nck), h(8);
+  JP_CUDA(cudaMemcpyAsync(hc.data(), cc, 24 * nck, cudaMemcpyDeviceToHost, st), "chunk D2H");
+  JP_CUDA(cudaMemcpyAsync(h.data(), at<int64_t>(ws, lo, R_HEADER), 64, cudaMemcpyDeviceToHost, st), "profile D2H");
+  JP_CUDA(cudaStreamSynchronize(st), "profile sync");
+  if (h[H_BAD]) return fail(JP_ERR_INDEX, "%lld index entries are outside their arrays", (long long)h[H_BAD]);
+  fill_profile(&res->prof, L->n, h.data());
+  res->profiled = 1;
+  // 2. chunk modes -> tasks (maximal same-mode runs)
+  struct Task { int64_t s, e; int mode; };
+  std::vector<Task> tasks;
+  for (int64_t k = 0; k < nck; k++) {
+    const int64_t s = k * chunk, e = std::min(L->n, s + chunk);
+    int m = select_mode_counts(e - s, hc[3 * k], hc[3 * k + 1], hc[3 * k + 2], c.tau_high);
+    if (m == JP_MODE_SEQ_RECOMMENDED) m = JP_MODE_TLS;
+    if (!tasks.empty() && tasks.back().mode == m) tasks.back().e = e;
+    else tasks.push_back({s, e, m});
+  }
+  // coarsen to <= 64 tasks: merge the smallest adjacent pair into the stronger mode
+  auto rank = [](int m) { return m == JP_MODE_TLS ? 2 : m == JP_MODE_PRIVATIZED ? 1 : 0; };
+  while ((int)tasks.size() > kMaxTasks) {
+    size_t best = 0;
+    for (size_t q = 1; q + 1 < tasks.size(); q++)
+      if (tasks[q].e - tasks[q].s + tasks[q + 1].e - tasks[q + 1].s <
+          tasks[best].e - tasks[best].s + tasks[best + 1].e - tasks[best + 1].s) best = q;
+    tasks[best].e = tasks[best + 1].e;
+    if (rank(tasks[best + 1].mode) > rank(tasks[best].mode)) tasks[best].mode = tasks[best + 1].mode;
+    tasks.erase(tasks.begin() + best + 1);
+  }
+  const int nt = (int)tasks.size();
+  res->n_tasks = nt;
+  res->mode = nt ? tasks[0].mode : JP_MODE_DOALL;
+  // 3. inter-task conflicts (PDG) and topological batches
+  std::vector<unsigned long long> conf(kMaxTasks, 0);
+  if (nt > 1) {
+    std::vector<int32_t> ct(nck);
+    for (int t = 0; t < nt; t++)
+      for (int64_t k = tasks[t].s / chunk; k * chunk < tasks[t].e; k++) ct[k] = t;
+    int32_t *dct = reinterpret_cast<int32_t *>(sch + sl.chunk_task);
+    JP_CUDA(cudaMemcpyAsync(dct, ct.data(), 4 * nck, cudaMemcpyHostToDevice, st), "task map H2D");
+    auto P = [&](size_t o) { return o == SIZE_MAX ? nullptr : reinterpret_cast<unsigned long long *>(sch + o); };
+    unsigned long long *dconf = P(sl.conf);
+    JP_CUDA(launch_task_conflicts(j, dct, chunk, P(sl.wmA), P(sl.rmA), P(sl.wmT), P(sl.rmT), dconf, st), "conflicts");
+    JP_CUDA(cudaMemcpyAsync(conf.data(), dconf, 8 * kMaxTasks, cudaMemcpyDeviceToHost, st), "conf D2H");
+    JP_CUDA(cudaStreamSynchronize(st), "conf sync");
+  }
+  std::vector<int> level(nt, 0);
+  int nlev = nt ? 1 : 0;
+  for (int u = 0; u < nt; u++) {
+    for (int t = 0; t < u; t++)
+      if ((conf[u] >> t) & 1ull) level[u] = std::max(level[u], level[t] + 1);
+    nlev = std::max(nlev, level[u] + 1);
+  }
+  res->n_batches = nlev;
+  // 4. run batch by batch; tasks of one batch are pairwise conflict-free and run
+  //    concurrently (TLS on one SM, partitioned modes on the rest)
+  int64_t *tstats = reinterpret_cast<int64_t *>(sch + sl.tstats);
+  cudaEvent_t ev0;
+  JP_CUDA(cudaEventCreateWithFlags(&ev0, cudaEventDisableTiming), "event");
+  std::vector<cudaEvent_t> evs;
+  std::vector<int> tls_tasks;
+  for (int lv = 0; lv < nlev; lv++) {
+    bool any_priv = false;
+    for (int t = 0; t < nt; t++) any_priv |= level[t] == lv && tasks[t].mode == JP_MODE_PRIVATIZED;
+    if (any_priv) {
+      if (lo.bytes[R_KEYS_A]) cudaMemsetAsync(at<char>(ws, lo, R_KEYS_A), 0, lo.bytes[R_KEYS_A], st);
+      if (lo.bytes[R_KEYS_T]) cudaMemsetAsync(at<char>(ws, lo, R_KEYS_T), 0, lo.bytes[R_KEYS_T], st);
+    }
+    cudaEventRecord(ev0, st);
+    int sidx = 0;
+    std::vector<cudaEvent_t> joins;
+    // TLS tasks first so that their single CTA is resident before the wide grids
+    for (int pass = 0; pass < 2; pass++) {
+      for (int t = 0; t < nt; t++) {
+        if (level[t] != lv) continue;
+        const bool tls = tasks[t].mode == JP_MODE_TLS;
+        if ((pass == 0) != tls) continue;
+        cudaStream_t s2 = g_pool.get(sidx++);
+        cudaStreamWaitEvent(s2, ev0, 0);
+        Job sj = sub_job(j, tasks[t].s, tasks[t].e);
+        if (tls) {
+          TlsPlan tp;
+          jp_tls_cfg tc{c.tls_window, c.tls_w_max, 1, 0};
+          jp_profile tprof{};
+          tprof.n = sj.d.n;
+          tprof.raw_iters = hc.empty() ? -1 : 0;
+          for (int64_t k = tasks[t].s / chunk; k * chunk < tasks[t].e; k++) { tprof.raw_iters += hc[3 * k]; tprof.waw_iters += hc[3 * k + 2]; }
+          JP_TRY(tls_plan(sj, &tc, &tprof, tp));
+          JP_CUDA(launch_tls(sj, ws, lo, tp, tstats + 4 * t, s2), "tls task");
+          tls_tasks.push_back(t);
+        } else if (tasks[t].mode == JP_MODE_PRIVATIZED) {
+          JP_CUDA(launch_priv_stream(sj, ws, lo, false, s2), "priv task");
+        } else {
+          JP_CUDA(launch_doall(sj, s2), "doall task");
+        }
+        res->task_mode_iters[tasks[t].mode] += sj.d.n;
+        cudaEvent_t e;
+        cudaEventCreateWithFlags(&e, cudaEventDisableTiming);
+        cudaEventRecord(e, s2);
+        joins.push_back(e);
+        evs.push_back(e);
+      }
+    }
+    for (auto e : joins) cudaStreamWaitEvent(st, e, 0);
+    if (any_priv) JP_CUDA(launch_priv_finalize(j, ws, lo, st), "priv finalize");
+  }
+  // stats of the TLS tasks
+  memset(&res->tls, 0, sizeof res->tls);
+  for (int t : tls_tasks) {
+    int64_t s4[4];
+    JP_CUDA(cudaMemcpyAsync(s4, tstats + 4 * t, sizeof s4, cudaMemcpyDeviceToHost, st), "tls stats D2H");
+    JP_CUDA(cudaStreamSynchronize(st), "tls stats sync");
+    res->tls.committed += s4[0]; res->tls.executed += s4[1]; res->tls.windows += s4[2]; res->tls.violations += s4[3];
+  }
+  JP_CUDA(cudaStreamSynchronize(st), "schedule sync");
+  cudaEventDestroy(ev0);
+  for (auto e : evs) cudaEventDestroy(e);
+  return JP_OK;
+}
+
+jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size_t ws_bytes, jp_sched_result *res,
+                      jp_stream_t stp) {
+  JP_TRY(check_loop(L));
+  if (!res) return fail(JP_ERR_ARG, "result is NULL");
+  JP_TRY(need_device());
+  jp_sched_cfg c = cfgp ? *cfgp : default_cfg();
+  if (c.tau_high <= 0.0) c.tau_high = 0.25;
+  if (c.chunk_iters <= 0) c.chunk_iters = 65536;
+  if (c.tls_w_max <= 0) c.tls_w_max = 4096;
+  memset(res, 0, sizeof *res);
+  cudaStream_t st = (cudaStream_t)stp;
+  Job j = make_job(L);
+  res->prof.n = L->n;
+  res->prof.first_raw_iter = -1;
+  if (!has_idx(j)) {   // "determined DOALL" (mode A): no profiling
+    res->mode = JP_MODE_DOALL;
+    res->profiled = 0;
+    res->n_tasks = 1;
+    res->n_batches = 1;
+    JP_CUDA(launch_doall(j, st), "doall");
+    res->task_mode_iters[JP_MODE_DOALL] = L->n;
+    return JP_OK;
+  }
+  if (c.scheme == JP_SCHED_STEALING) return schedule_stealing(L, j, c, ws, ws_bytes, res, st);
+  if (c.scheme != JP_SCHED_SHARING) return fail(JP_ERR_ARG, "bad scheme %d", c.scheme);
+  jp_profile p;
+  JP_TRY(jp_profile_density(L, ws, ws_bytes, nullptr, 0, nullptr, &p, stp));
+  res->prof = p;
+  res->profiled = 1;
+  res->mode = select_mode_counts(p.n, p.raw_iters, p.war_iters, p.waw_iters, c.tau_high);
+  res->n_tasks = 1;
+  res->n_batches = 1;
+  const int run = res->mode == JP_MODE_SEQ_RECOMMENDED ? JP_MODE_TLS : res->mode;
+  return run_mode(L, j, run, &p, c, ws, ws_bytes, res, st);
+}
+
+// ---------------------------------------------------------------------------
+// host-buffer entry point (end-to-end: H2D, schedule, D2H)
+// ---------------------------------------------------------------------------
+struct Stage { size_t off[7]; size_t total; };
+static Stage stage_layout(const jp_loop *L) {
+  Stage s{};
+  bool ur, ur2, uw, us;
+  used_idx(L->op, ur, ur2, uw, us);
+  const size_t sz[7] = {(ur && L->r) ? 4 * (size_t)L->n : 0, (ur2 && L->r2) ? 4 * (size_t)L->n : 0,
+                        (uw && L->w) ? 4 * (size_t)L->n : 0, (us && L->s) ? 4 * (size_t)L->n : 0,
+                        4 * (size_t)L->len_A, L->X ? 4 * (size_t)L->len_X : 0, L->T ? 4 * (size_t)L->len_T : 0};
+  size_t o = 0;
+  for (int k = 0; k < 7; k++) { s.off[k] = sz[k] ? o : SIZE_MAX; o = al256(o + sz[k]); }
+  s.total = o;
+  return s;
+}
+
+size_t jp_stage_bytes(const jp_loop *L) {
+  if (!L || check_loop(L) == JP_ERR_ARG) return 0;
+  return stage_layout(L).total;
+}
+
+jp_status jp_schedule_host(const jp_loop *Lh, const jp_sched_cfg *cfg, void *stage, size_t stage_bytes, void *ws,
+                           size_t ws_bytes, jp_sched_result *res, jp_stream_t stp) {
+  JP_TRY(check_loop(Lh));
+  JP_TRY(need_device());
+  Stage sl = stage_layout(Lh);
+  if (!stage || stage_bytes < sl.total) return fail(JP_ERR_WORKSPACE, "stage buffer needs %zu bytes", sl.total);
+  cudaStream_t st = (cudaStream_t)stp;
+  jp_loop Ld = *Lh;
+  char *b = static_cast<char *>(stage);
+  const void *src[7] = {Lh->r, Lh->r2, Lh->w, Lh->s, Lh->A, Lh->X, Lh->T};
+  const size_t sz[7] = {4 * (size_t)Lh->n, 4 * (size_t)Lh->n, 4 * (size_t)Lh->n, 4 * (size_t)Lh->n,
+                        4 * (size_t)Lh->len_A, 4 * (size_t)Lh->len_X, 4 * (size_t)Lh->len_T};
+  void *dst[7];
+  for (int k = 0; k < 7; k++) {
+    dst[k] = sl.off[k] == SIZE_MAX ? nullptr : b + sl.off[k];
+    if (dst[k] && sz[k]) JP_CUDA(cudaMemcpyAsync(dst[k], src[k], sz[k], cudaMemcpyHostToDevice, st), "stage H2D");
+  }
+  Ld.r = (const int32_t *)dst[0]; Ld.r2 = (const int32_t *)dst[1]; Ld.w = (const int32_t *)dst[2];
+  Ld.s = (const int32_t *)dst[3]; Ld.A = dst[4]; Ld.X = dst[5]; Ld.T = dst[6];
+  JP_TRY(jp_schedule(&Ld, cfg, ws, ws_bytes, res, stp));
+  if (Lh->len_A) JP_CUDA(cudaMemcpyAsync(Lh->A, Ld.A, sz[4], cudaMemcpyDeviceToHost, st), "stage D2H");
+  if (Lh->T && Lh->len_T && Lh->op == JP_OP_PRIV_TMP)
+    JP_CUDA(cudaMemcpyAsync(Lh->T, Ld.T, sz[6], cudaMemcpyDeviceToHost, st), "stage D2H");
+  JP_CUDA(cudaStreamSynchronize(st), "stage sync");
+  return JP_OK;
+}
+
+}  // extern "C"

@@ -1,0 +1,74 @@
+// jp_host.h -- host-side internals of libjp.so (workspace layout, launchers).
+#pragma once
+#include <cstddef>
+#include <cstdint>
+#include <cuda_runtime.h>
+#include "jp_internal.cuh"
+
+namespace jp {
+
+enum Region : int {
+  R_HEADER = 0, R_MINW_A = 1, R_MINR_A = 2, R_MINW_T = 3, R_MINR_T = 4, R_KEYS_A = 5,
+  R_KEYS_T = 6, R_TLS_S_A = 7, R_TLS_C_A = 8, R_TLS_S_T = 9, R_TLS_C_T = 10, R_SCHED = 11,
+  R_COUNT = 12
+};
+
+struct Layout {
+  size_t off[R_COUNT];
+  size_t bytes[R_COUNT];
+  size_t total;
+};
+
+// Fixed-offset layout of a workspace for loop L (offsets do not depend on uses).
+Layout layout(const jp_loop *L);
+// End of the furthest region the JP_WS_* uses touch.
+size_t layout_end(const Layout &lo, int uses);
+constexpr int64_t kSchedMinChunk = 1024;
+constexpr int kMaxTasks = 64;
+// scheduler scratch sub-layout (inside R_SCHED)
+struct SchedLayout {
+  size_t counts, chunk_task, wmA, rmA, wmT, rmT, conf, tstats, total;
+};
+SchedLayout sched_layout(const jp_loop *L);
+
+template <typename T> inline T *at(void *ws, const Layout &lo, int r) {
+  return lo.bytes[r] ? reinterpret_cast<T *>(static_cast<char *>(ws) + lo.off[r]) : nullptr;
+}
+
+// A (sub-)loop ready to launch: the device view plus its opcode and dtype.
+struct Job {
+  DLoop d;
+  int op, dt;
+};
+Job make_job(const jp_loop *L);
+
+// ---- launchers (each returns the first CUDA error, if any) ----
+cudaError_t launch_validate(const Job &j, int64_t *hdr, cudaStream_t st);
+cudaError_t launch_prof_stamp(const Job &j, void *ws, const Layout &lo, cudaStream_t st);
+cudaError_t launch_prof_classify(const Job &j, void *ws, const Layout &lo, uint32_t *raw_bits,
+                                 int64_t chunk, int64_t *chunk_counts, cudaStream_t st);
+cudaError_t launch_doall(const Job &j, cudaStream_t st, int max_ctas = 0);
+cudaError_t launch_priv_stream(const Job &j, void *ws, const Layout &lo, bool clear_keys,
+                               cudaStream_t st, int max_ctas = 0);
+cudaError_t launch_priv_finalize(const Job &j, void *ws, const Layout &lo, cudaStream_t st);
+cudaError_t launch_merge_apply(void *arr, int64_t len, const int64_t *keys, cudaStream_t st);
+// STEALING scheduler helpers (jp_sched.cu): per-task write/read bitmasks of every
+// address, then the task x task conflict matrix conf[t] (bit u set: t and u
+// touch a common address and at least one of them writes it).
+cudaError_t launch_task_conflicts(const Job &j, const int32_t *chunk_task, int64_t chunk,
+                                  unsigned long long *wmA, unsigned long long *rmA,
+                                  unsigned long long *wmT, unsigned long long *rmT,
+                                  unsigned long long *conf, cudaStream_t st);
+
+struct TlsPlan {
+  int64_t window, w_max, prof_raw;  // prof_raw < 0: no profile
+  bool waw;                         // in-window WAW resolution needed
+  int path;                         // 1 cta, 2 grid
+};
+// stats: int64[4] device (committed, executed, windows, violations); bar: u32[2]
+// zeroed barrier words + int64[3] fv slots (grid path).
+cudaError_t launch_tls(const Job &j, void *ws, const Layout &lo, const TlsPlan &p, int64_t *stats,
+                       cudaStream_t st);
+int64_t tls_next_window(int64_t n, int64_t prof_raw, int64_t prev_commit, int64_t w_max);
+
+}  // namespace jp

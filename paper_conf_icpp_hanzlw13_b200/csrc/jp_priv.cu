@@ -1,0 +1,205 @@
+// jp_priv.cu -- privatized execution PE(V) (the
+// private(list) clause, Table I: "a copy of each variable in list is
+// allocated for each execution element").
+//
+// Reading A10: exposed reads see the pre-loop values (legal iff d_raw = 0),
+// the covered read of T sees the iteration's own private value (a register).
+// Reading A9: after all iterations every address holds the value of its
+// highest-gid writer -- realised with packed keys (gid+1)<<32 | bits(v) and
+// atomicMax, so it composes across CTAs and (via an int64 MAX all-reduce)
+// across GPUs.  Arrays reached only through identity indices are stored
+// directly (one writer per address, no key).
+//
+// Hot-address handling (config 4 writes 2^26 values into 1024 slots): small
+// keyed arrays get a per-CTA shared table of the highest local iteration that
+// wrote each slot.  Each CTA walks its iterations in DESCENDING order, so the
+// first touch of a slot is already its CTA-local last writer and every later
+// touch fails the plain shared-memory check without issuing an atomic; the
+// flush then recomputes the winner's value and issues one 64-bit global
+// atomicMax per (CTA, touched slot).
+#include "jp_host.h"
+
+namespace jp {
+
+constexpr int kPrivThreads = 512;
+
+__device__ __forceinline__ void smem_last(uint32_t *tab, int64_t a, int64_t i) {
+  const uint32_t v = (uint32_t)(i + 1);
+  if (tab[a] < v) atomicMax(&tab[a], v);
+}
+
+template <int OP, int DT>
+__global__ void __launch_bounds__(kPrivThreads) k_priv_generic(DLoop L, unsigned long long *kA,
+                                                                unsigned long long *kT, int smA, int smT) {
+  extern __shared__ uint32_t sm[];
+  uint32_t *tA = smA ? sm : nullptr;
+  uint32_t *tT = smT ? sm + (smA ? L.lenA : 0) : nullptr;
+  const int64_t ns = (smA ? L.lenA : 0) + (smT ? L.lenT : 0);
+  for (int64_t k = threadIdx.x; k < ns; k += blockDim.x) sm[k] = 0;
+  __syncthreads();
+  const int64_t stride = (int64_t)gridDim.x * blockDim.x;
+  for (int64_t j = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; j < L.n; j += stride) {
+    const int64_t i = L.n - 1 - j;          // descending within every CTA
+    uint32_t va = 0, vt = 0;
+    body_values<OP, DT>(L, i, L.A, va, vt);  // A is untouched until finalize when keyed
+    const int64_t a = ixl(L, L.w, i);
+    if (kA) {
+      if (tA) smem_last(tA, a, i);
+      else atomicMax(&kA[a], pack_key(L.base + i, va));
+    } else {
+      L.A[a] = va;
+    }
+    if constexpr (OP == JP_OP_PRIV_TMP) {
+      const int64_t b = ixl(L, L.s, i);
+      if (kT) {
+        if (tT) smem_last(tT, b, i);
+        else atomicMax(&kT[b], pack_key(L.base + i, vt));
+      } else {
+        L.T[b] = vt;
+      }
+    }
+  }
+  __syncthreads();
+  if (tA) {
+    for (int64_t a = threadIdx.x; a < L.lenA; a += blockDim.x) {
+      const uint32_t e = tA[a];
+      if (e) {
+        uint32_t va = 0, vt = 0;
+        body_values<OP, DT>(L, e - 1, L.A, va, vt);
+        atomicMax(&kA[a], pack_key(L.base + e - 1, va));
+      }
+    }
+  }
+  if (tT) {
+    for (int64_t b = threadIdx.x; b < L.lenT; b += blockDim.x) {
+      const uint32_t e = tT[b];
+      if (e) {
+        uint32_t va = 0, vt = 0;
+        body_values<OP, DT>(L, e - 1, L.A, va, vt);
+        atomicMax(&kT[b], pack_key(L.base + e - 1, vt));
+      }
+    }
+  }
+}
+
+// PRIV_TMP with r = w = NULL, s indirect, small T (config 4): 16-byte lanes.
+// Per iteration: X 4 B + s 4 B read, Y 4 B written (12 B/iter algorithmic).
+template <int DT>
+__global__ void __launch_bounds__(kPrivThreads) k_priv_tmp_vec(DLoop L, unsigned long long *kT, int64_t nvec) {
+  extern __shared__ uint32_t tT[];
+  for (int64_t k = threadIdx.x; k < L.lenT; k += blockDim.x) tT[k] = 0;
+  __syncthreads();
+  const uint4 *X4 = reinterpret_cast<const uint4 *>(L.X);
+  const int4 *S4 = reinterpret_cast<const int4 *>(L.s);
+  uint4 *Y4 = reinterpret_cast<uint4 *>(L.A);
+  constexpr int U = 2;
+  const int64_t stride = (int64_t)gridDim.x * blockDim.x * U;
+  for (int64_t j0 = (int64_t)blockIdx.x * blockDim.x * U + threadIdx.x; j0 < nvec; j0 += stride) {
+    uint4 x[U];
+    int4 s[U];
+#pragma unroll
+    for (int u = 0; u < U; u++) {
+      const int64_t j = j0 + (int64_t)u * blockDim.x;
+      if (j < nvec) {
+        const int64_t v = nvec - 1 - j;
+        x[u] = __ldcs(X4 + v);
+        s[u] = __ldcs(S4 + v);
+      }
+    }
+#pragma unroll
+    for (int u = 0; u < U; u++) {
+      const int64_t j = j0 + (int64_t)u * blockDim.x;
+      if (j < nvec) {
+        const int64_t v = nvec - 1 - j;
+        uint4 y;
+        y.x = op_add<DT>(op_mul<DT>(L.c0, x[u].x), L.c1);
+        y.y = op_add<DT>(op_mul<DT>(L.c0, x[u].y), L.c1);
+        y.z = op_add<DT>(op_mul<DT>(L.c0, x[u].z), L.c1);
+        y.w = op_add<DT>(op_mul<DT>(L.c0, x[u].w), L.c1);
+        __stcs(Y4 + v, y);
+        smem_last(tT, s[u].w, 4 * v + 3);
+        smem_last(tT, s[u].z, 4 * v + 2);
+        smem_last(tT, s[u].y, 4 * v + 1);
+        smem_last(tT, s[u].x, 4 * v + 0);
+      }
+    }
+  }
+  if (blockIdx.x == 0) {  // scalar tail [4*nvec, n)
+    for (int64_t i = 4 * nvec + threadIdx.x; i < L.n; i += blockDim.x) {
+      const uint32_t t = op_mul<DT>(L.c0, L.X[i]);
+      L.A[i] = op_add<DT>(t, L.c1);
+      smem_last(tT, L.s[i], i);
+    }
+  }
+  __syncthreads();
+  for (int64_t b = threadIdx.x; b < L.lenT; b += blockDim.x) {
+    const uint32_t e = tT[b];
+    if (e) atomicMax(&kT[b], pack_key(L.base + e - 1, op_mul<DT>(L.c0, L.X[e - 1])));
+  }
+}
+
+__global__ void k_apply_keys(uint32_t *arr, int64_t len, const unsigned long long *keys) {
+  const int64_t stride = (int64_t)gridDim.x * blockDim.x;
+  for (int64_t a = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; a < len; a += stride) {
+    const unsigned long long k = keys[a];
+    if (k) arr[a] = (uint32_t)k;   // written only where some iteration wrote (safe beside concurrent tasks)
+  }
+}
+
+static bool al16(const void *p) { return ((uintptr_t)p & 15) == 0; }
+
+template <int OP, int DT>
+static void run_priv(const DLoop &d, unsigned long long *kA, unsigned long long *kT, cudaStream_t st, int max_ctas) {
+  int grid = num_sms() * 2;
+  if (max_ctas > 0 && grid > max_ctas) grid = max_ctas;
+  if constexpr (OP == JP_OP_PRIV_TMP) {
+    if (!d.r && !d.w && d.s && d.ioff == 0 && kT && !kA && d.lenT <= kSmemSlots && al16(d.X) && al16(d.s) &&
+        al16(d.A)) {
+      int64_t nvec = d.n / 4;
+      int64_t need = (nvec + kPrivThreads * 2 - 1) / (kPrivThreads * 2);
+      if (need < grid) grid = (int)(need < 1 ? 1 : need);
+      k_priv_tmp_vec<DT><<<grid, kPrivThreads, d.lenT * 4, st>>>(d, kT, nvec);
+      note_launch();
+      return;
+    }
+  }
+  int smA = kA && d.lenA <= kSmemSlots, smT = kT && d.lenT <= kSmemSlots;
+  size_t smem = ((smA ? d.lenA : 0) + (smT ? d.lenT : 0)) * 4;
+  int64_t need = (d.n + kPrivThreads - 1) / kPrivThreads;
+  if (need < grid) grid = (int)(need < 1 ? 1 : need);
+  k_priv_generic<OP, DT><<<grid, kPrivThreads, smem, st>>>(d, kA, kT, smA, smT);
+  note_launch();
+}
+
+cudaError_t launch_priv_stream(const Job &j, void *ws, const Layout &lo, bool clear_keys, cudaStream_t st,
+                               int max_ctas) {
+  auto *kA = at<unsigned long long>(ws, lo, R_KEYS_A);
+  auto *kT = at<unsigned long long>(ws, lo, R_KEYS_T);
+  if (clear_keys) {
+    if (kA) cudaMemsetAsync(kA, 0, lo.bytes[R_KEYS_A], st);
+    if (kT) cudaMemsetAsync(kT, 0, lo.bytes[R_KEYS_T], st);
+  }
+  if (j.d.n == 0) return launch_check();
+  JP_DISPATCH(j.op, j.dt, run_priv, j.d, kA, kT, st, max_ctas);
+  return launch_check();
+}
+
+static void apply(uint32_t *arr, int64_t len, const unsigned long long *keys, cudaStream_t st) {
+  if (!len || !keys) return;
+  int64_t need = (len + 255) / 256, cap = (int64_t)num_sms() * 8;
+  k_apply_keys<<<(int)(need < cap ? need : cap), 256, 0, st>>>(arr, len, keys);
+  note_launch();
+}
+
+cudaError_t launch_priv_finalize(const Job &j, void *ws, const Layout &lo, cudaStream_t st) {
+  apply(j.d.A, j.d.lenA, at<unsigned long long>(ws, lo, R_KEYS_A), st);
+  if (j.op == JP_OP_PRIV_TMP) apply(j.d.T, j.d.lenT, at<unsigned long long>(ws, lo, R_KEYS_T), st);
+  return launch_check();
+}
+
+cudaError_t launch_merge_apply(void *arr, int64_t len, const int64_t *keys, cudaStream_t st) {
+  apply(static_cast<uint32_t *>(arr), len, reinterpret_cast<const unsigned long long *>(keys), st);
+  return launch_check();
+}
+
+}  // namespace jp

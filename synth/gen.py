@@ -55,15 +55,20 @@ def permutation(seed: int, n: int, device="cpu", stream: int = 7) -> torch.Tenso
     return torch.argsort(keys, stable=True)
 
 
-def i32_data(seed: int, stream: int, n: int, device="cpu") -> torch.Tensor:
-    """A0[k] = rnd(seed, stream, k) & 0xFFFFF   (int32)."""
-    return (rnd(seed, stream, _ar(n, device)) & 0xFFFFF).to(torch.int32)
+def i32_data(seed: int, stream: int, n: int, device="cpu", start: int = 0) -> torch.Tensor:
+    """A0[k] = rnd(seed, stream, k) & 0xFFFFF   (int32), k in [start, start+n)."""
+    return (rnd(seed, stream, _ar(n, device, start)) & 0xFFFFF).to(torch.int32)
 
 
-def f32_data(seed: int, stream: int, n: int, device="cpu") -> torch.Tensor:
-    """X[k] = (rnd >> 41) * 2^-22 - 1: uniform on [-1, 1) on a 2^-22 grid, exact in fp32."""
-    m = _lsr(rnd(seed, stream, _ar(n, device)), 41).to(torch.float64)
-    return (m * (2.0 ** -22) - 1.0).to(torch.float32)
+def f32_data(seed: int, stream: int, n: int, device="cpu", start: int = 0) -> torch.Tensor:
+    """X[k] = (rnd >> 41) * 2^-22 - 1: uniform on [-1, 1) on a 2^-22 grid, exact in fp32.
+    Generated in slices so that 2^28-element arrays fit comfortably."""
+    out = torch.empty(n, dtype=torch.float32, device=device)
+    step = 1 << 24
+    for o in range(0, n, step):
+        m = _lsr(rnd(seed, stream, _ar(min(step, n - o), device, start + o)), 41).to(torch.float64)
+        out[o:o + step] = (m * (2.0 ** -22) - 1.0).to(torch.float32)
+    return out
 
 
 def dependent_set(seed: int, n: int, k: int, device="cpu") -> torch.Tensor:
@@ -137,11 +142,14 @@ def config1(density: float = 0.05, n: int = 4096, delta: int = 64, device="cpu")
                     meta={"raw": k, "war": 0, "waw": 0, "delta": delta, "density": density})
 
 
-def config2(n: int = 1 << 28, device="cpu") -> Workload:
-    """Config 2: DOALL streaming SAXPY fp32, affine (r = w = NULL)."""
+def config2(n: int = 1 << 28, device="cpu", start: int = 0, count: int | None = None) -> Workload:
+    """Config 2: DOALL streaming SAXPY fp32, affine (r = w = NULL).  start/count
+    select a shard [start, start+count) of the n-iteration loop (task sharing)."""
     seed = 1002
-    return Workload("config2", 1, 1, n, f32_data(seed, 6, n, device), X=f32_data(seed, 2, n, device),
-                    c0=C0_F32, meta={"raw": 0, "war": 0, "waw": 0})
+    count = n - start if count is None else count
+    return Workload("config2", 1, 1, count, f32_data(seed, 6, count, device, start),
+                    X=f32_data(seed, 2, count, device, start), c0=C0_F32,
+                    meta={"raw": 0, "war": 0, "waw": 0, "start": start, "total": n})
 
 
 def config3(density: float = 0.01, n: int = 1 << 24, delta: int = 1024, device="cpu") -> Workload:

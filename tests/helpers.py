@@ -1,0 +1,62 @@
+"""Shared test helpers: workload <-> oracle/jp conversions and random loops."""
+from __future__ import annotations
+
+import numpy as np
+import torch
+
+import oracle as O
+import synth
+
+
+def to_oracle(wl) -> O.Loop:
+    a = lambda t: None if t is None else t.cpu().numpy()  # noqa: E731
+    return O.Loop(wl.op, wl.dtype, wl.n, a(wl.A), r=a(wl.r), r2=a(wl.r2), w=a(wl.w), s=a(wl.s), X=a(wl.X),
+                  T=a(wl.T), c0=wl.c0, c1=wl.c1)
+
+
+def random_loop(seed: int, op: int, dtype: int, n: int, len_a: int | None = None, null_prob=0.2,
+                dup_writes=True, slots=None) -> synth.Workload:
+    """Random loop of any opcode; lengths are chosen so identity indices stay in range."""
+    g = np.random.default_rng(seed)
+    # decide which index arrays are NULL first: identity accesses need len >= n
+    null = {k: g.random() < null_prob for k in ("r", "w", "r2", "s")}
+    a_ident = (null["w"] or (op in (O.OP_ADD_C, O.OP_STENCIL2) and null["r"])
+               or (op == O.OP_STENCIL2 and null["r2"]))
+    la = len_a if len_a is not None else max(n, 8)
+    if a_ident:
+        la = max(la, n)
+    lx = max(n, 8)
+    lt = slots or max(8, n // 16)
+    if op == O.OP_PRIV_TMP and null["s"]:
+        lt = max(lt, n)
+    el = np.int32 if dtype == O.I32 else np.float32
+
+    def idx(key, hi):
+        if null[key]:
+            return None
+        if dup_writes or hi < n:
+            return torch.from_numpy(g.integers(0, hi, size=n).astype(np.int32))
+        return torch.from_numpy(g.permutation(hi)[:n].astype(np.int32))
+
+    def data(m):
+        if dtype == O.I32:
+            return torch.from_numpy(g.integers(-2**31, 2**31, size=m, dtype=np.int64).astype(np.int32))
+        return torch.from_numpy(((g.integers(0, 2**23, size=m) * 2.0**-22) - 1).astype(el))
+
+    r = idx("r", lx if op in (O.OP_SAXPY, O.OP_PRIV_TMP) else la)
+    w = idx("w", la)
+    r2 = idx("r2", la) if op == O.OP_STENCIL2 else None
+    s = idx("s", lt) if op == O.OP_PRIV_TMP else None
+    c0 = np.float32(1.1) if dtype == O.F32 else 7
+    c1 = np.float32(0.3) if dtype == O.F32 else -3
+    return synth.Workload("random", op, dtype, n, data(la), r=r, r2=r2, w=w, s=s,
+                          X=data(lx) if op in (O.OP_SAXPY, O.OP_PRIV_TMP) else None,
+                          T=data(lt) if op == O.OP_PRIV_TMP else None, c0=float(c0), c1=float(c1))
+
+
+def bits_to_flags(raw_bits: torch.Tensor, n: int) -> np.ndarray:
+    b = raw_bits.cpu().numpy().view(np.uint32)
+    out = np.zeros(n, dtype=np.uint8)
+    for k in range(n):
+        out[k] = (b[k >> 5] >> (k & 31)) & 1
+    return out

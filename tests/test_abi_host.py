@@ -1,0 +1,185 @@
+"""CPU-side checks of the C ABI (-m "not gpu"): libjp.so loads, exports every
+symbol include/jp.h declares, and its host-only logic (workspace layout, the
+Fig. 2(b) decision, the task-sharing / task-stealing plans) matches the plain
+restatements in oracle/sched.py.  No compute call is made without a GPU, except
+to check that one fails loudly with JP_ERR_CUDA (no CPU fallback)."""
+import os
+import random
+import re
+
+import pytest
+import torch
+
+import oracle.sched as S
+import paper_conf_icpp_hanzlw13_b200 as jp
+from paper_conf_icpp_hanzlw13_b200 import _abi
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+
+
+def header_functions():
+    src = open(os.path.join(ROOT, "include", "jp.h")).read()
+    src = re.sub(r"/\*.*?\*/", "", src, flags=re.S)
+    return sorted(set(re.findall(r"\b(jp_[a-z_]+)\s*\(", src)))
+
+
+def test_library_exports_every_header_symbol():
+    lib = jp.lib()
+    names = header_functions()
+    assert len(names) >= 20
+    for name in names:
+        assert hasattr(lib, name), name
+    assert sorted(n for n, _, _ in _abi.SIGNATURES) == names
+
+
+def test_version_and_launch_counter():
+    assert "sm_100a" in jp.jp_version()
+    assert jp.jp_launch_count() >= 0
+
+
+def cpu_loop(op=0, n=1000, la=1000, r=True, w=True, s=False, lt=16):
+    A = torch.zeros(la, dtype=torch.int32)
+    idx = torch.zeros(n, dtype=torch.int32)
+    return jp.Loop(op, 0, n, A, r=idx if r else None, w=idx if w else None, s=idx if s else None,
+                   X=torch.zeros(max(n, 8), dtype=torch.int32) if op in (1, 2) else None,
+                   T=torch.zeros(lt, dtype=torch.int32) if op == 2 else None)
+
+
+def test_workspace_layout_fixed_offsets():
+    L = cpu_loop()
+    sizes = {u: jp.jp_workspace_bytes(L, u) for u in (0, 1, 2, 4, 8, 15)}
+    assert sizes[0] == 4096
+    assert sizes[1] < sizes[2] < sizes[4] < sizes[8] == sizes[15]
+    # regions are disjoint, 256-aligned and inside the total
+    spans = []
+    for name in _abi.REGIONS:
+        off, nb = jp.jp_ws_region(L, name)
+        assert off % 256 == 0
+        if nb:
+            spans.append((off, off + nb))
+            assert off + nb <= sizes[15]
+    spans.sort()
+    for a, b in zip(spans, spans[1:]):
+        assert a[1] <= b[0]
+    # identity-only arrays need no tables
+    La = cpu_loop(r=False, w=False)
+    assert jp.jp_ws_region(La, "minW_A")[1] == 0 and jp.jp_ws_region(La, "keys_A")[1] == 0
+    Lt = cpu_loop(op=2, r=False, w=False, s=True, lt=1024)
+    assert jp.jp_ws_region(Lt, "minW_T")[1] == 4 * 1024 and jp.jp_ws_region(Lt, "keys_T")[1] == 8 * 1024
+    assert jp.jp_ws_region(Lt, "keys_A")[1] == 0
+
+
+@pytest.mark.parametrize("seed", range(200))
+def test_select_mode_matches_fig2b(seed):
+    g = random.Random(seed)
+    n = g.choice([1, 100, 4096])
+    raw = g.choice([0, 0, 1, n // 100, n // 10, n // 3, n])
+    war, waw = g.choice([0, 0, 5]), g.choice([0, 0, 7])
+    all_null = g.random() < 0.15
+    L = cpu_loop(r=not all_null, w=not all_null)
+    p = {"n": n, "raw_iters": raw, "war_iters": war, "waw_iters": waw, "first_raw_iter": -1,
+         "d_raw": raw / n, "d_war": war / n, "d_waw": waw / n}
+    tau = g.choice([0.25, 0.05, 0.5])
+    assert jp.jp_select_mode(L, p, tau) == S.select_mode(all_null, n, raw, war, waw, tau)
+
+
+def test_select_mode_paper_cases():
+    """P:L624-629 (BlackScholes, DD ~ 0.012 -> GPU-TLS, mode B)
+    (CFD/Sepia: no TD, some FD -> mode D); P:L611-613 (Gauss-Seidel, high -> C)."""
+    L = cpu_loop()
+    mk = lambda n, r, a, b: {"n": n, "raw_iters": r, "war_iters": a, "waw_iters": b, "first_raw_iter": -1,  # noqa
+                             "d_raw": r / n, "d_war": a / n, "d_waw": b / n}
+    assert jp.jp_select_mode(L, mk(1000, 12, 0, 0)) == jp.JP_MODE_TLS
+    assert jp.jp_select_mode(L, mk(1000, 0, 900, 900)) == jp.JP_MODE_PRIVATIZED
+    assert jp.jp_select_mode(L, mk(1000, 999, 999, 0)) == jp.JP_MODE_SEQ_RECOMMENDED
+    assert jp.jp_select_mode(L, mk(1000, 0, 0, 0)) == jp.JP_MODE_DOALL
+    assert jp.jp_select_mode(cpu_loop(r=False, w=False), None) == jp.JP_MODE_DOALL
+
+
+def test_boundary_formula_paper_hardware():
+    """P:L354-358 with the paper's platform: 12 cores at 2.66 GHz
+    and 448 GPU cores; the M2050 clock 1.15 GHz is NOT in the paper (external)."""
+    b = S.boundary(448, 1.15, 12, 2.66)
+    assert abs(b - 515.2 / 547.12) < 1e-12
+    n = 10_000_000
+    rg = jp.jp_plan_sharing(n, 2, [448 * 1.15, 12 * 2.66])
+    assert rg[0] == (0, int(n * b)) and rg[1] == (int(n * b), n)
+
+
+@pytest.mark.parametrize("seed", range(50))
+def test_plan_sharing_matches_oracle(seed):
+    g = random.Random(seed)
+    world = g.randint(1, 8)
+    n = g.choice([0, 1, 7, 1 << 28, g.randint(0, 10**9)])
+    weights = None if g.random() < 0.3 else [g.uniform(0.1, 5.0) for _ in range(world)]
+    got = jp.jp_plan_sharing(n, world, weights)
+    assert got == S.sharing_ranges(n, weights or [1.0] * world)
+    assert got[0][0] == 0 and got[-1][1] == n
+    for a, b in zip(got, got[1:]):
+        assert a[1] == b[0]
+    if weights is None and n % world == 0:
+        assert all(e - s == n // world for s, e in got)   # closed form 1/k on identical GPUs
+
+
+@pytest.mark.parametrize("seed", range(60))
+def test_plan_stealing_matches_oracle(seed):
+    g = random.Random(seed)
+    world = g.randint(1, 8)
+    pos, tasks = 0, []
+    for _ in range(g.randint(1, 6)):
+        ln = g.randint(1, 50000)
+        tasks.append((pos, pos + ln, g.choice([0, 0, 1, 2])))
+        pos += ln
+    chunk = g.choice([1024, 4096, 65536])
+    speed = None if g.random() < 0.4 else [g.uniform(0.5, 3.0) for _ in range(world)]
+    st = g.uniform(0.01, 1.0)
+    got, stolen = jp.jp_plan_stealing(tasks, world, chunk, speed, st)
+    exp, estolen = S.stealing_plan(tasks, world, chunk, speed, st)
+    assert got == exp and stolen == estolen
+    # every iteration of every task is owned exactly once; TLS stays on rank 0
+    cover = sorted((c[0], c[1]) for c in got)
+    assert cover[0][0] == 0 and cover[-1][1] == pos
+    for a, b in zip(cover, cover[1:]):
+        assert a[1] == b[0]
+    assert all(c[3] == 0 for c in got if c[2] == 2)
+    assert all(0 <= c[3] < world for c in got)
+
+
+def test_stealing_bicg_mechanism():
+    """P:L633-641 (BICG): eight equal sub-loops all land in one queue at first;
+    the empty worker gets one and then steals.  Two equal-speed workers here:
+    the mechanism (dealing + tail stealing) must leave both busy.  The paper's
+    62.5% CPU share depends on unreported speeds: parity unpinned."""
+    tasks = [(k * 1000, (k + 1) * 1000, 0) for k in range(8)]
+    chunks, stolen = jp.jp_plan_stealing(tasks, 2, 1000, [1.0, 1.0], 1.0)
+    owners = [c[3] for c in chunks]
+    assert owners.count(0) == owners.count(1) == 4 and stolen == 0
+    chunks, stolen = jp.jp_plan_stealing(tasks, 2, 1000, [3.0, 1.0], 1.0)
+    owners = [c[3] for c in chunks]
+    assert owners.count(0) > owners.count(1)   # faster worker ends up with more sub-loops
+    # a TLS task pinned to rank 0 makes rank 1 steal rank 0's DOALL chunks
+    tasks = [(0, 8000, 2)] + [(8000 + k * 1000, 9000 + k * 1000, 0) for k in range(8)]
+    chunks, stolen = jp.jp_plan_stealing(tasks, 2, 1000, [1.0, 1.0], 1.0)
+    assert stolen >= 3 and sum(1 for c in chunks if c[3] == 1) >= 7
+
+
+@pytest.mark.skipif(torch.cuda.is_available(), reason="checks the no-GPU failure path")
+def test_compute_calls_fail_loudly_without_gpu():
+    L = cpu_loop()
+    with pytest.raises(jp.JPError) as e:
+        jp.jp_run_doall(L)
+    assert e.value.status == _abi.JP_ERR_CUDA
+    with pytest.raises(jp.JPError) as e:
+        jp.jp_schedule(L, torch.zeros(1 << 20, dtype=torch.uint8))
+    assert e.value.status == _abi.JP_ERR_CUDA
+
+
+def test_bad_arguments():
+    with pytest.raises(jp.JPError) as e:
+        jp.jp_plan_sharing(10, 2, [0.0, 0.0])
+    assert e.value.status == _abi.JP_ERR_ARG
+    A = torch.zeros(10, dtype=torch.int32)
+    L = jp.Loop(0, 0, 11, A)          # identity index past len_A
+    with pytest.raises(jp.JPError) as e:
+        jp.jp_ws_region(L, "header")
+    assert e.value.status == _abi.JP_ERR_INDEX

@@ -1,0 +1,462 @@
+"""GPU parity: every mode of libjp.so against the CPU oracle (bit-exact).
+
+Run on a B200 with ``pytest -m gpu``.  Every call goes through the C ABI
+(paper_conf_icpp_hanzlw13_b200 -> libjp.so); the expected values come only from
+oracle/ (test infrastructure) on the same seeded inputs.  Tolerance: none --
+int32 bodies wrap and fp32 bodies are two separately rounded RN ops compiled
+with -fmad=false on both sides (BASELINE.json north_star; reading A12), so the
+bar is byte equality of every output array and exact integer statistics.
+"""
+import itertools
+
+import numpy as np
+import pytest
+import torch
+
+import oracle as O
+import synth
+from helpers import bits_to_flags, random_loop, to_oracle
+
+pytestmark = pytest.mark.gpu
+
+if torch.cuda.is_available():
+    import paper_conf_icpp_hanzlw13_b200 as jp
+    DEV = torch.device("cuda:0")
+else:  # collected on CPU boxes, never run there
+    jp = None
+    DEV = None
+
+OPS = [O.OP_ADD_C, O.OP_SAXPY, O.OP_PRIV_TMP, O.OP_STENCIL2]
+DTS = [O.I32, O.F32]
+
+
+def gpu(wl):
+    return wl.to(DEV)
+
+
+def same(t: torch.Tensor, a: np.ndarray) -> bool:
+    return t.cpu().numpy().tobytes() == a.tobytes()
+
+
+def check_arrays(g, A, T):
+    assert same(g.A, A), f"A differs at {np.flatnonzero(g.A.cpu().numpy() != A)[:10]}"
+    if T is not None:
+        assert same(g.T, T), f"T differs at {np.flatnonzero(g.T.cpu().numpy() != T)[:10]}"
+
+
+# ---------------------------------------------------------------------------
+# profiler
+# ---------------------------------------------------------------------------
+def prof_case(wl):
+    ref = O.profile(to_oracle(wl))
+    g = gpu(wl)
+    L = jp.Loop.from_workload(g)
+    ws = jp.workspace(L, jp.JP_WS_PROFILE)
+    bits = torch.zeros((wl.n + 31) // 32 + 1, dtype=torch.int32, device=DEV)
+    p = jp.jp_profile_density(L, ws, raw_bits=bits)
+    assert (p["raw_iters"], p["war_iters"], p["waw_iters"]) == (ref["raw_iters"], ref["war_iters"], ref["waw_iters"])
+    assert p["first_raw_iter"] == ref["first_raw_iter"]
+    assert np.array_equal(bits_to_flags(bits, wl.n), ref["flags"] & 1)
+    return p, ref
+
+
+@pytest.mark.parametrize("op,dt,seed", [(op, dt, s) for op in OPS for dt in DTS for s in range(3)])
+def test_profile_random(op, dt, seed):
+    n = [1, 37, 1000, 4099][seed % 4] if seed < 3 else 5000
+    wl = random_loop(1000 * op + 10 * dt + seed, op, dt, n + 17 * seed, len_a=max(64, (n + 17 * seed) // 3))
+    prof_case(wl)
+
+
+@pytest.mark.parametrize("d", [0.0, 0.05])
+def test_profile_config1(d):
+    p, _ = prof_case(synth.config1(d))
+    assert p["raw_iters"] == (205 if d else 0)
+
+
+@pytest.mark.parametrize("d", [0.001, 0.01, 0.05, 0.10])
+def test_profile_config3_reduced(d):
+    prof_case(synth.config3(d, n=(1 << 18) + 5))
+
+
+def test_profile_config4_and_5():
+    prof_case(synth.config4(n=(1 << 18) + 3))
+    prof_case(synth.config5(n=1 << 16))
+
+
+def test_profile_chunk_counts():
+    wl = synth.config5(n=1 << 16)
+    ref = O.profile(to_oracle(wl))
+    g = gpu(wl)
+    L = jp.Loop.from_workload(g)
+    ws = jp.workspace(L)
+    chunk = 1024
+    cc = torch.full((wl.n // chunk * 3,), -7, dtype=torch.int64, device=DEV)
+    jp.jp_profile_density(L, ws, chunk_iters=chunk, chunk_counts=cc)
+    cc = cc.cpu().numpy().reshape(-1, 3)
+    f = ref["flags"].reshape(-1, chunk)
+    assert np.array_equal(cc[:, 0], (f & 1).sum(1))
+    assert np.array_equal(cc[:, 1], ((f >> 1) & 1).sum(1))
+    assert np.array_equal(cc[:, 2], ((f >> 2) & 1).sum(1))
+
+
+def test_profile_partitioned_equals_whole():
+    """C1: stamp each rank's range with global ids, MAX-combine the int32 tables,
+    classify each range; the summed counts equal the single-GPU profile."""
+    wl = synth.config3(0.05, n=1 << 16)
+    ref = O.profile(to_oracle(wl))
+    g = gpu(wl)
+    k = 3
+    rg = jp.jp_plan_sharing(wl.n, k)
+    loops, wss = [], []
+    for (s, e) in rg:
+        L = jp.Loop(g.op, g.dtype, e - s, g.A, r=g.r[s:e], w=g.w[s:e], c0=g.c0, iter_base=s)
+        loops.append(L)
+        wss.append(jp.workspace(L, jp.JP_WS_PROFILE))
+        jp.jp_profile_stamp(L, wss[-1])
+    torch.cuda.synchronize()
+    for reg in ("minW_A", "minR_A"):
+        off, nb = jp.jp_ws_region(loops[0], reg)
+        views = [w[off:off + nb].view(torch.int32) for w in wss]
+        m = views[0].clone()
+        for v in views[1:]:
+            m = torch.maximum(m, v)
+        for v in views:
+            v.copy_(m)
+    tot = [0, 0, 0]
+    for L, w in zip(loops, wss):
+        p = jp.jp_profile_classify(L, w)
+        tot = [tot[0] + p["raw_iters"], tot[1] + p["war_iters"], tot[2] + p["waw_iters"]]
+    assert tot == [ref["raw_iters"], ref["war_iters"], ref["waw_iters"]]
+
+
+def test_index_error_no_side_effects():
+    wl = synth.config1(0.05)
+    wl.w[100] = 4096   # out of range
+    g = gpu(wl)
+    A0 = g.A.clone()
+    L = jp.Loop.from_workload(g)
+    ws = jp.workspace(L)
+    with pytest.raises(jp.JPError) as e:
+        jp.jp_profile_density(L, ws)
+    assert e.value.status == -5
+    for fn in (lambda: jp.jp_run_doall(L, None, ws), lambda: jp.jp_run_privatized(L, None, ws),
+               lambda: jp.jp_run_tls(L, 256, ws=ws), lambda: jp.jp_schedule(L, ws)):
+        with pytest.raises(jp.JPError) as e:
+            fn()
+        assert e.value.status == -5
+    torch.cuda.synchronize()
+    assert torch.equal(g.A, A0)
+    assert jp.jp_validate(L, ws) == 1
+
+
+def test_illegal_modes_and_workspace():
+    wl = synth.config1(0.05)
+    g = gpu(wl)
+    L = jp.Loop.from_workload(g)
+    ws = jp.workspace(L)
+    p = jp.jp_profile_density(L, ws)
+    with pytest.raises(jp.JPError) as e:
+        jp.jp_run_doall(L, p, ws)
+    assert e.value.status == -4
+    with pytest.raises(jp.JPError) as e:
+        jp.jp_run_privatized(L, p, ws)
+    assert e.value.status == -4
+    small = torch.empty(1024, dtype=torch.uint8, device=DEV)
+    with pytest.raises(jp.JPError) as e:
+        jp.jp_profile_density(L, small)
+    assert e.value.status == -3
+
+
+# ---------------------------------------------------------------------------
+# DOALL
+# ---------------------------------------------------------------------------
+@pytest.mark.parametrize("op,dt", list(itertools.product(OPS, DTS)))
+def test_doall_affine(op, dt):
+    n = (1 << 20) + 3
+    wl = random_loop(77 + op * 2 + dt, op, dt, n, null_prob=1.0)   # all indices NULL
+    _, A, T = O.run_seq(to_oracle(wl))
+    g = gpu(wl)
+    res = jp.jp_schedule(jp.Loop.from_workload(g))
+    assert res["mode"] == jp.JP_MODE_DOALL and res["profiled"] == 0
+    torch.cuda.synchronize()
+    check_arrays(g, A, T)
+
+
+def test_doall_misaligned_scalar_path():
+    n = 4099
+    wl = synth.config2(n=n + 1)
+    g = gpu(wl)
+    A_off, X_off = g.A[1:], g.X[1:]         # 4-byte offset: not 16-byte aligned
+    ref = O.Loop(1, 1, n, wl.A[1:].numpy(), X=wl.X[1:].numpy(), c0=wl.c0)
+    exp = O.run_seq(ref)[1]
+    jp.jp_run_doall(jp.Loop(1, 1, n, A_off, X=X_off, c0=wl.c0))
+    torch.cuda.synchronize()
+    assert same(A_off, exp)
+
+
+@pytest.mark.parametrize("op,dt", list(itertools.product(OPS, DTS)))
+def test_doall_indirect_permutation(op, dt):
+    n = 50000
+    g0 = np.random.default_rng(op * 10 + dt)
+    wl = random_loop(5 + op * 2 + dt, op, dt, n, len_a=n, dup_writes=False, null_prob=0.0, slots=n)
+    pi = torch.from_numpy(g0.permutation(n).astype(np.int32))
+    wl.w = pi
+    if op in (O.OP_ADD_C,):
+        wl.r = pi
+    if op == O.OP_STENCIL2:
+        wl.r, wl.r2 = pi, pi
+    if op == O.OP_PRIV_TMP:
+        wl.s = torch.from_numpy(g0.permutation(n).astype(np.int32))
+    ref = to_oracle(wl)
+    p = O.profile(ref)
+    assert (p["raw_iters"], p["war_iters"], p["waw_iters"]) == (0, 0, 0)
+    _, A, T = O.run_seq(ref)
+    g = gpu(wl)
+    L = jp.Loop.from_workload(g)
+    res = jp.jp_schedule(L, jp.workspace(L))
+    assert res["mode"] == jp.JP_MODE_DOALL and res["profiled"] == 1
+    torch.cuda.synchronize()
+    check_arrays(g, A, T)
+
+
+def test_config2_full_size_sampled():
+    """BASELINE size N=2^28 in the bench's launch configuration; outputs sampled
+    and recomputed one by one by the oracle."""
+    n = 1 << 28
+    wl = synth.config2(n=n, device=DEV)
+    Y0 = wl.A.clone()
+    jp.jp_schedule(jp.Loop.from_workload(wl))
+    torch.cuda.synchronize()
+    idx = torch.cat([torch.arange(0, 4096), torch.randint(0, n, (1 << 16,), generator=torch.Generator().manual_seed(1)),
+                     torch.arange(n - 4096, n)]).to(DEV)
+    x, y0, y = wl.X[idx].cpu().numpy(), Y0[idx].cpu().numpy(), wl.A[idx].cpu().numpy()
+    ref = O.Loop(1, 1, len(idx), y0, X=x, c0=wl.c0)
+    assert y.tobytes() == O.run_seq(ref)[1].tobytes()
+
+
+# ---------------------------------------------------------------------------
+# privatized
+# ---------------------------------------------------------------------------
+@pytest.mark.parametrize("n", [1, 31, 4096 + 7, (1 << 20) + 5])
+def test_priv_config4(n):
+    wl = synth.config4(n=n)
+    ref = to_oracle(wl)
+    _, A, T = O.run_seq(ref)
+    _, A2, T2 = O.sim_priv(ref)
+    assert A.tobytes() == A2.tobytes() and T.tobytes() == T2.tobytes()
+    g = gpu(wl)
+    L = jp.Loop.from_workload(g)
+    ws = jp.workspace(L)
+    res = jp.jp_schedule(L, ws)
+    torch.cuda.synchronize()
+    if n > 1024 + 64:
+        assert res["mode"] == jp.JP_MODE_PRIVATIZED
+    check_arrays(g, A, T)
+
+
+@pytest.mark.parametrize("op,dt,seed", [(op, dt, s) for op in OPS for dt in DTS for s in range(2)])
+def test_priv_random_raw_free(op, dt, seed):
+    """Random loops made RAW-free by construction: exposed reads only from
+    addresses no iteration writes (or identity/self)."""
+    n = 20000 + seed * 4097
+    wl = random_loop(300 + op * 10 + dt * 3 + seed, op, dt, n, len_a=2 * n, null_prob=0.1,
+                     slots=[7, 3000][seed])
+    g0 = np.random.default_rng(seed)
+    if wl.w is not None:
+        wl.w = torch.from_numpy(g0.integers(0, n, size=n).astype(np.int32))      # writes in [0, n): WAW
+    if op in (O.OP_ADD_C, O.OP_STENCIL2):
+        wl.r = torch.from_numpy(g0.integers(n, 2 * n, size=n).astype(np.int32))  # reads in [n, 2n)
+        if op == O.OP_STENCIL2:
+            wl.r2 = torch.from_numpy(g0.integers(n, 2 * n, size=n).astype(np.int32))
+        if wl.w is None:
+            wl.w = torch.from_numpy(g0.integers(0, n, size=n).astype(np.int32))
+    if op == O.OP_SAXPY and wl.w is not None:
+        wl.w = torch.from_numpy(g0.permutation(2 * n)[:n].astype(np.int32))     # Y read = write: must be unique
+    ref = to_oracle(wl)
+    p = O.profile(ref)
+    assert p["raw_iters"] == 0
+    _, A, T = O.run_seq(ref)
+    g = gpu(wl)
+    L = jp.Loop.from_workload(g)
+    ws = jp.workspace(L)
+    jp.jp_run_privatized(L, None, ws)
+    torch.cuda.synchronize()
+    check_arrays(g, A, T)
+
+
+def test_priv_split_merge_equals_whole():
+    """C4: two ranges privatized into separate key tables, int64 MAX-combined,
+    applied once -- equals the sequential result (global last writer)."""
+    wl = synth.config4(n=(1 << 18) + 9)
+    _, A, T = O.run_seq(to_oracle(wl))
+    g = gpu(wl)
+    rg = jp.jp_plan_sharing(wl.n, 2)
+    keys = []
+    for (s, e) in rg:
+        L = jp.Loop(g.op, g.dtype, e - s, g.A[s:e], s=g.s[s:e], X=g.X[s:e], T=g.T, c0=g.c0, c1=g.c1, iter_base=s)
+        ws = jp.workspace(L, jp.JP_WS_PRIV)
+        jp.jp_priv_stream(L, {"n": e - s, "raw_iters": 0, "war_iters": 1, "waw_iters": 1, "first_raw_iter": -1,
+                              "d_raw": 0.0, "d_war": 0.0, "d_waw": 0.0}, ws)
+        off, nb = jp.jp_ws_region(L, "keys_T")
+        keys.append(ws[off:off + nb].view(torch.int64))
+    torch.cuda.synchronize()
+    merged = torch.maximum(keys[0], keys[1])
+    jp.jp_merge_apply(g.T, merged)
+    torch.cuda.synchronize()
+    check_arrays(g, A, T)
+
+
+def test_config4_full_size():
+    """BASELINE size N=2^26 (bench launch configuration), compared in full."""
+    wl = synth.config4()
+    _, A, T = O.run_seq(to_oracle(wl))
+    g = gpu(wl)
+    L = jp.Loop.from_workload(g)
+    ws = jp.workspace(L)
+    res = jp.jp_schedule(L, ws)
+    torch.cuda.synchronize()
+    assert res["mode"] == jp.JP_MODE_PRIVATIZED
+    check_arrays(g, A, T)
+
+
+# ---------------------------------------------------------------------------
+# TLS
+# ---------------------------------------------------------------------------
+def tls_case(wl, window, path, w_max=65536, with_prof=False):
+    ref = to_oracle(wl)
+    prof_raw = O.profile(ref)["raw_iters"] if with_prof else -1
+    st, A, T, stats = O.sim_tls(ref, window, w_max, prof_raw)
+    g = gpu(wl)
+    L = jp.Loop.from_workload(g)
+    ws = jp.workspace(L)
+    p = jp.jp_profile_density(L, ws) if with_prof else None
+    got = jp.jp_run_tls(L, window=window, w_max=w_max, path=path, prof=p, ws=ws)
+    torch.cuda.synchronize()
+    check_arrays(g, A, T)
+    assert got == stats, (got, stats)
+    return got
+
+
+@pytest.mark.parametrize("window,path", [(32, 1), (100, 1), (1024, 1), (4096, 1), (32, 2), (1000, 2), (8192, 2),
+                                         (65536, 2)])
+@pytest.mark.parametrize("d", [0.0, 0.05])
+def test_tls_config1(window, path, d):
+    tls_case(synth.config1(d), window, path)
+
+
+@pytest.mark.parametrize("d", [0.001, 0.01, 0.10])
+@pytest.mark.parametrize("path", [1, 2])
+def test_tls_config3_reduced(d, path):
+    tls_case(synth.config3(d, n=(1 << 17) + 11), 4096, path)
+
+
+@pytest.mark.parametrize("op,dt,seed", [(op, dt, s) for op in OPS for dt in DTS for s in range(3)])
+def test_tls_random(op, dt, seed):
+    n = [200, 3000, 9001][seed]
+    wl = random_loop(500 + op * 10 + dt * 3 + seed, op, dt, n, len_a=max(32, n // [1, 4, 2][seed]))
+    for window, path in ((64, 1), (1000, 1), (1000, 2)):
+        if op == O.OP_PRIV_TMP and window > 2048 and path == 1:
+            continue
+        tls_case(wl, window, path)
+
+
+@pytest.mark.parametrize("path", [1, 2])
+def test_tls_adaptive(path):
+    wl = synth.config3(0.01, n=1 << 16)
+    w_max = 4096 if path == 1 else 65536
+    tls_case(wl, 0, path, w_max=w_max, with_prof=True)
+    tls_case(synth.config3(0.05, n=1 << 16), 0, path, w_max=w_max, with_prof=False)
+
+
+def test_tls_gauss_seidel_and_prefix_chain():
+    n = 3000
+    A0 = torch.arange(n, dtype=torch.int32)
+    ar = torch.arange(n, dtype=torch.int32)
+    gs = synth.Workload("gs", 3, 0, n, A0.clone(), r=torch.clamp(ar - 1, min=0), r2=torch.clamp(ar + 1, max=n - 1),
+                        w=ar.clone(), c0=3)
+    st = tls_case(gs, 256, 1)
+    assert st["windows"] == n and st["violations"] == n - 1
+    pc = synth.Workload("pc", 0, 0, n, A0.clone(), r=torch.clamp(ar - 1, min=0), w=ar.clone(), c0=7)
+    st = tls_case(pc, 1000, 2)
+    assert st["windows"] == n and st["violations"] == n - 1
+
+
+def test_config3_full_size_stats():
+    """BASELINE size N=2^24 at d=1%, W=4096 (bench configuration): full arrays and stats."""
+    tls_case(synth.config3(0.01), 4096, 1)
+
+
+# ---------------------------------------------------------------------------
+# scheduler
+# ---------------------------------------------------------------------------
+def test_schedule_modes_fig2b():
+    cases = [(synth.config1(0.0), jp.JP_MODE_DOALL), (synth.config1(0.05), jp.JP_MODE_TLS),
+             (synth.config4(n=1 << 14), jp.JP_MODE_PRIVATIZED)]
+    n = 2048
+    ar = torch.arange(n, dtype=torch.int32)
+    gs = synth.Workload("gs", 3, 0, n, torch.arange(n, dtype=torch.int32), r=torch.clamp(ar - 1, min=0),
+                        r2=torch.clamp(ar + 1, max=n - 1), w=ar.clone(), c0=3)
+    cases.append((gs, jp.JP_MODE_SEQ_RECOMMENDED))
+    for wl, mode in cases:
+        _, A, T = O.run_seq(to_oracle(wl))
+        g = gpu(wl)
+        L = jp.Loop.from_workload(g)
+        res = jp.jp_schedule(L, jp.workspace(L))
+        assert res["mode"] == mode, (wl.name, res)
+        torch.cuda.synchronize()
+        check_arrays(g, A, T)
+
+
+@pytest.mark.parametrize("n,chunk", [(1 << 16, 1024), ((1 << 18), 4096)])
+def test_schedule_stealing_config5(n, chunk):
+    wl = synth.config5(n=n)
+    _, A, T = O.run_seq(to_oracle(wl))
+    g = gpu(wl)
+    L = jp.Loop.from_workload(g)
+    res = jp.jp_schedule(L, jp.workspace(L), scheme=jp.JP_SCHED_STEALING, chunk_iters=chunk)
+    torch.cuda.synchronize()
+    check_arrays(g, A, T)
+    assert res["task_mode_iters"][jp.JP_MODE_DOALL] == n // 2
+    assert res["task_mode_iters"][jp.JP_MODE_TLS] == n // 4
+    assert res["task_mode_iters"][jp.JP_MODE_PRIVATIZED] == n // 4
+    assert res["n_batches"] == 1
+
+
+def test_schedule_stealing_dependent_tasks():
+    """Tasks that share addresses must be ordered (2MM/Crypt-style dependent batches)."""
+    n, chunk = 1 << 14, 1024
+    ar = torch.arange(n, dtype=torch.int32)
+    r = ar.clone()
+    w = ar.clone()
+    # second half reads what the first half wrote, far back (RAW across tasks, TLS-free inside)
+    r[n // 2:] = ar[: n // 2]
+    w[n // 2:] = ar[n // 2:]
+    wl = synth.Workload("dep", 0, 0, n, torch.arange(n, dtype=torch.int32) * 3, r=r, w=w, c0=5)
+    _, A, T = O.run_seq(to_oracle(wl))
+    g = gpu(wl)
+    L = jp.Loop.from_workload(g)
+    res = jp.jp_schedule(L, jp.workspace(L), scheme=jp.JP_SCHED_STEALING, chunk_iters=chunk)
+    torch.cuda.synchronize()
+    check_arrays(g, A, T)
+
+
+def test_schedule_host_e2e():
+    wl = synth.config1(0.05)
+    _, A, _ = O.run_seq(to_oracle(wl))
+    h = {k: (v.pin_memory() if v is not None else None) for k, v in wl.arrays().items()}
+    L = jp.Loop(wl.op, wl.dtype, wl.n, h["A"], r=h["r"], w=h["w"], c0=wl.c0)
+    stage = torch.empty(jp.jp_stage_bytes(L), dtype=torch.uint8, device=DEV)
+    Ld = jp.Loop.from_workload(gpu(wl))
+    ws = jp.workspace(Ld)
+    res = jp.jp_schedule_host(L, stage, ws)
+    assert res["mode"] == jp.JP_MODE_TLS
+    assert h["A"].numpy().tobytes() == A.tobytes()
+
+
+def test_launch_count_and_version():
+    n0 = jp.jp_launch_count()
+    g = gpu(synth.config2(n=4096))
+    jp.jp_schedule(jp.Loop.from_workload(g))
+    torch.cuda.synchronize()
+    assert jp.jp_launch_count() == n0 + 1
+    assert "sm_100a" in jp.jp_version()
