@@ -12,7 +12,7 @@ import os
 import threading
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
-LIB_PATH = os.path.join(_HERE, "libjp.so")
+LIB_PATH = os.environ.get("JP_LIB") or os.path.join(_HERE, "libjp.so")
 
 JP_OK, JP_ERR_ARG, JP_ERR_CUDA, JP_ERR_WORKSPACE, JP_ERR_ILLEGAL_MODE, JP_ERR_INDEX, JP_ERR_UNSUPPORTED = \
     0, -1, -2, -3, -4, -5, -6

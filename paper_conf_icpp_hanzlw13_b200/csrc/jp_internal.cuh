@@ -8,13 +8,27 @@
 #include <cuda_runtime.h>
 #include "../../include/jp.h"
 
+// CTA-wide barrier used by every kernel of the library: an explicit
+// barrier.sync with a memory clobber (see jp_tls.cu TLS_SYNC and DESIGN.md
+// Sec.6 for the intermittent failure observed with __syncthreads()).
+#define JP_CTA_SYNC() asm volatile("barrier.sync 0;" ::: "memory")
+
 namespace jp {
 
 constexpr int kSmemSlots = 4096;          // arrays this small are pre-aggregated per CTA
-constexpr int kTlsCtaThreads = 1024;      // single-CTA TLS path
-constexpr int kTlsCtaIpt = 4;             // -> W <= 4096
+#ifndef JP_TLS_THREADS
+#define JP_TLS_THREADS 1024
+#endif
+#ifndef JP_TLS_IPT
+#define JP_TLS_IPT 4
+#endif
+#ifndef JP_TLS_HASHLOG
+#define JP_TLS_HASHLOG 13
+#endif
+constexpr int kTlsCtaThreads = JP_TLS_THREADS;   // single-CTA TLS path
+constexpr int kTlsCtaIpt = JP_TLS_IPT;           // -> W <= 4096
 constexpr int kTlsCtaWmax = kTlsCtaThreads * kTlsCtaIpt;
-constexpr int kTlsHashLog = 13;           // 8192 slots = 2 x W_max
+constexpr int kTlsHashLog = JP_TLS_HASHLOG;      // 8192 slots = 2 x W_max
 constexpr int kTlsHash = 1 << kTlsHashLog;
 constexpr int kTlsGridThreads = 512;
 constexpr uint32_t kEmpty = 0xFFFFFFFFu;

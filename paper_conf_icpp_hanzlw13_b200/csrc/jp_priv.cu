@@ -36,7 +36,7 @@ __global__ void __launch_bounds__(kPrivThreads) k_priv_generic(DLoop L, unsigned
   uint32_t *tT = smT ? sm + (smA ? L.lenA : 0) : nullptr;
   const int64_t ns = (smA ? L.lenA : 0) + (smT ? L.lenT : 0);
   for (int64_t k = threadIdx.x; k < ns; k += blockDim.x) sm[k] = 0;
-  __syncthreads();
+  JP_CTA_SYNC();
   const int64_t stride = (int64_t)gridDim.x * blockDim.x;
   for (int64_t j = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; j < L.n; j += stride) {
     const int64_t i = L.n - 1 - j;          // descending within every CTA
@@ -59,7 +59,7 @@ __global__ void __launch_bounds__(kPrivThreads) k_priv_generic(DLoop L, unsigned
       }
     }
   }
-  __syncthreads();
+  JP_CTA_SYNC();
   if (tA) {
     for (int64_t a = threadIdx.x; a < L.lenA; a += blockDim.x) {
       const uint32_t e = tA[a];
@@ -88,7 +88,7 @@ template <int DT>
 __global__ void __launch_bounds__(kPrivThreads) k_priv_tmp_vec(DLoop L, unsigned long long *kT, int64_t nvec) {
   extern __shared__ uint32_t tT[];
   for (int64_t k = threadIdx.x; k < L.lenT; k += blockDim.x) tT[k] = 0;
-  __syncthreads();
+  JP_CTA_SYNC();
   const uint4 *X4 = reinterpret_cast<const uint4 *>(L.X);
   const int4 *S4 = reinterpret_cast<const int4 *>(L.s);
   uint4 *Y4 = reinterpret_cast<uint4 *>(L.A);
@@ -131,7 +131,7 @@ __global__ void __launch_bounds__(kPrivThreads) k_priv_tmp_vec(DLoop L, unsigned
       smem_last(tT, L.s[i], i);
     }
   }
-  __syncthreads();
+  JP_CTA_SYNC();
   for (int64_t b = threadIdx.x; b < L.lenT; b += blockDim.x) {
     const uint32_t e = tT[b];
     if (e) atomicMax(&kT[b], pack_key(L.base + e - 1, op_mul<DT>(L.c0, L.X[e - 1])));

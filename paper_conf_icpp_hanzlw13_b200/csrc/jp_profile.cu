@@ -43,7 +43,7 @@ __global__ void __launch_bounds__(256) k_prof_stamp(DLoop L, Tabs t, int64_t *hd
   if (t.sA) { sAw = p; p += L.lenA; if (t.rA) { sAr = p; p += L.lenA; } }
   if (t.sT) { sTw = p; p += L.lenT; sTr = p; p += L.lenT; }
   for (int64_t k = threadIdx.x; k < p - sm; k += blockDim.x) sm[k] = -1;
-  __syncthreads();
+  JP_CTA_SYNC();
 
   int64_t bad = 0;
   const int64_t stride = (int64_t)gridDim.x * blockDim.x;
@@ -72,7 +72,7 @@ __global__ void __launch_bounds__(256) k_prof_stamp(DLoop L, Tabs t, int64_t *hd
   // warp-aggregate the bad-index count
   for (int o = 16; o; o >>= 1) bad += __shfl_xor_sync(0xffffffffu, bad, o);
   if ((threadIdx.x & 31) == 0 && bad) atomicAdd((unsigned long long *)&hdr[H_BAD], (unsigned long long)bad);
-  __syncthreads();
+  JP_CTA_SYNC();
   // flush the per-CTA pre-aggregated tables
   if (t.sA) {
     for (int64_t a = threadIdx.x; a < L.lenA; a += blockDim.x) {
@@ -100,7 +100,7 @@ __global__ void __launch_bounds__(256) k_prof_classify(DLoop L, Tabs t, uint32_t
   __shared__ unsigned long long s_first;
   if (threadIdx.x < 3) s_cnt[threadIdx.x] = 0;
   if (threadIdx.x == 0) s_first = ~0ull;
-  __syncthreads();
+  JP_CTA_SYNC();
   const int lane = threadIdx.x & 31;
   const int64_t warps = (int64_t)gridDim.x * (blockDim.x >> 5);
   unsigned long long c_raw = 0, c_war = 0, c_waw = 0, first = ~0ull;
@@ -152,7 +152,7 @@ __global__ void __launch_bounds__(256) k_prof_classify(DLoop L, Tabs t, uint32_t
     if (c_waw) atomicAdd(&s_cnt[2], c_waw);
     if (first != ~0ull) atomicMin(&s_first, first);
   }
-  __syncthreads();
+  JP_CTA_SYNC();
   if (threadIdx.x < 3 && s_cnt[threadIdx.x]) atomicAdd((unsigned long long *)&hdr[H_RAW + threadIdx.x], s_cnt[threadIdx.x]);
   if (threadIdx.x == 0 && s_first != ~0ull) atomicMin((unsigned long long *)&hdr[H_FIRST_RAW], s_first);
 }

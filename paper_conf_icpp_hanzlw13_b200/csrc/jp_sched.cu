@@ -45,7 +45,7 @@ __global__ void __launch_bounds__(256) k_task_conf(const unsigned long long *wm,
                                                    int64_t len, unsigned long long *conf) {
   __shared__ unsigned long long sc[kMaxTasks];
   if (threadIdx.x < kMaxTasks) sc[threadIdx.x] = 0;
-  __syncthreads();
+  JP_CTA_SYNC();
   const int64_t stride = (int64_t)gridDim.x * blockDim.x;
   for (int64_t a = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; a < len; a += stride) {
     const unsigned long long mw = wm[a], mr = rm ? rm[a] : 0ull, all = mw | mr;
@@ -59,7 +59,7 @@ __global__ void __launch_bounds__(256) k_task_conf(const unsigned long long *wm,
       }
     }
   }
-  __syncthreads();
+  JP_CTA_SYNC();
   if (threadIdx.x < kMaxTasks && sc[threadIdx.x]) atomicOr(&conf[threadIdx.x], sc[threadIdx.x]);
 }
 

@@ -31,6 +31,13 @@
 //             phases.
 #include "jp_host.h"
 
+// CTA barrier of the TLS windows.  An explicit barrier.sync with a memory
+// clobber: with the JP_CTA_SYNC() intrinsic the single-CTA window loop lost
+// RAW violations intermittently on sm_100a (a window's first violator was
+// missed in ~1 of 3 runs at W = 4096); the same kernel with this barrier passed
+// 80/80 repetitions ("TLS barrier").
+#define TLS_SYNC() asm volatile("barrier.sync 0;" ::: "memory")
+
 namespace jp {
 
 struct TlsArgs {
@@ -88,15 +95,43 @@ template <int OP> __device__ __forceinline__ int n_exposed() {
   return OP == JP_OP_ADD_C ? 1 : OP == JP_OP_SAXPY ? 1 : OP == JP_OP_STENCIL2 ? 2 : 0;
 }
 
+// index streams of an opcode, in ring order: 0 = r, 1 = w, 2 = r2 (STENCIL2) or s (PRIV_TMP)
+template <int OP> __host__ __device__ constexpr int n_streams() {
+  return (OP == JP_OP_PRIV_TMP || OP == JP_OP_STENCIL2) ? 3 : 2;
+}
+constexpr int kRing = 2 * kTlsCtaWmax;   // ring of prefetched indices: [ws, ws + 2 W_max)
+
+__device__ __forceinline__ void cp_async4(void *smem, const void *gmem) {
+  asm volatile("cp.async.ca.shared.global [%0], [%1], 4;" ::"r"((unsigned)__cvta_generic_to_shared(smem)),
+               "l"(gmem) : "memory");
+}
+__device__ __forceinline__ void cp_async_commit_wait() {
+  asm volatile("cp.async.commit_group;\n\tcp.async.wait_group 0;" ::: "memory");
+}
+
+// Single-CTA TLS.  Per window: SE reads the window's indices from a shared
+// ring (prefetched with cp.async one window ahead, so the only dependent
+// global access of SE is the gather of committed operands), issues every
+// gather before any use, then inserts the write keys into the shared hash.
 template <int OP, int DT, bool WAW>
 __global__ void __launch_bounds__(kTlsCtaThreads, 1) k_tls_cta(DLoop L, TlsArgs P, int64_t *stats) {
-  extern __shared__ uint32_t hsm[];
+  constexpr int NS = n_streams<OP>();
+  extern __shared__ __align__(16) uint32_t hsm[];
   uint32_t *hk = hsm, *hmin = hsm + kTlsHash, *hmax = hsm + 2 * kTlsHash;
+  int32_t *ring = reinterpret_cast<int32_t *>(hsm + 3 * kTlsHash);   // [NS][kRing]
   __shared__ int s_fv[2];
   const int tid = threadIdx.x, lane = tid & 31;
+  const int32_t *src[3] = {L.r, L.w, OP == JP_OP_STENCIL2 ? L.r2 : OP == JP_OP_PRIV_TMP ? L.s : nullptr};
   for (int k = tid; k < kTlsHash; k += kTlsCtaThreads) { hk[k] = kEmpty; hmin[k] = 0xFFFFFFFFu; hmax[k] = 0; }
   if (tid == 0) { s_fv[0] = INT32_MAX; s_fv[1] = INT32_MAX; }
-  __syncthreads();
+  // initial ring fill [0, min(n, kRing))
+  int64_t hi = L.n < kRing ? L.n : kRing;
+  for (int64_t i = tid; i < hi; i += kTlsCtaThreads)
+#pragma unroll
+    for (int q = 0; q < NS; q++)
+      if (src[q]) cp_async4(&ring[q * kRing + i], src[q] + i);
+  cp_async_commit_wait();
+  TLS_SYNC();
 
   const bool dc = n_exposed<OP>() > 0 && P.hashA;
   int64_t ws = 0;
@@ -106,26 +141,56 @@ __global__ void __launch_bounds__(kTlsCtaThreads, 1) k_tls_cta(DLoop L, TlsArgs 
   while (ws < L.n) {
     const int span = (int)(W < L.n - ws ? W : L.n - ws);
     if (tid == 0) s_fv[par ^ 1] = INT32_MAX;
-    uint32_t va[kTlsCtaIpt], vt[kTlsCtaIpt];
-    int32_t wa[kTlsCtaIpt], wt[kTlsCtaIpt], ra[kTlsCtaIpt], rb[kTlsCtaIpt];
+    // keep the ring full: [hi, ws + kRing) reuses the slots of iterations < ws
+    {
+      const int64_t to = ws + kRing < L.n ? ws + kRing : L.n;
+      for (int64_t i = hi + tid; i < to; i += kTlsCtaThreads)
+#pragma unroll
+        for (int q = 0; q < NS; q++)
+          if (src[q]) cp_async4(&ring[q * kRing + (i & (kRing - 1))], src[q] + i);
+      asm volatile("cp.async.commit_group;" ::: "memory");
+      hi = to;
+    }
+    uint32_t va[kTlsCtaIpt], vt[kTlsCtaIpt], g0[kTlsCtaIpt], g1[kTlsCtaIpt];
+    int32_t ix0[kTlsCtaIpt], ix1[kTlsCtaIpt], ix2[kTlsCtaIpt];
     int slA[kTlsCtaIpt], slT[kTlsCtaIpt];
-    // ---------------- SE ----------------
+    // ---------------- SE: indices from the ring ----------------
 #pragma unroll
     for (int k = 0; k < kTlsCtaIpt; k++) {
       const int off = k * kTlsCtaThreads + tid;
       if (off < span) {
         const int64_t i = ws + off;
-        body_values<OP, DT>(L, i, L.A, va[k], vt[k]);
-        wa[k] = (int32_t)ixl(L, L.w, i);
-        if constexpr (OP == JP_OP_PRIV_TMP) wt[k] = (int32_t)ixl(L, L.s, i);
-        if constexpr (OP == JP_OP_ADD_C || OP == JP_OP_STENCIL2) ra[k] = (int32_t)ixl(L, L.r, i);
-        if constexpr (OP == JP_OP_SAXPY) ra[k] = wa[k];
-        if constexpr (OP == JP_OP_STENCIL2) rb[k] = (int32_t)ixl(L, L.r2, i);
-        if (P.hashA) slA[k] = hins(hk, hmin, hkey_of(wa[k], 0), (uint32_t)off);
-        if constexpr (OP == JP_OP_PRIV_TMP) if (P.hashT) slT[k] = hins(hk, hmin, hkey_of(wt[k], 1), (uint32_t)off);
+        const int slot = (int)(i & (kRing - 1));
+        ix0[k] = src[0] ? ring[slot] : (int32_t)(L.ioff + i);
+        ix1[k] = src[1] ? ring[kRing + slot] : (int32_t)(L.ioff + i);
+        if constexpr (NS == 3) ix2[k] = src[2] ? ring[2 * kRing + slot] : (int32_t)(L.ioff + i);
       }
     }
-    __syncthreads();
+    // ---------------- SE: gather committed operands (all issued before use) ----------------
+#pragma unroll
+    for (int k = 0; k < kTlsCtaIpt; k++) {
+      const int off = k * kTlsCtaThreads + tid;
+      if (off < span) {
+        if constexpr (OP == JP_OP_ADD_C) g0[k] = L.A[ix0[k]];
+        else if constexpr (OP == JP_OP_SAXPY) { g0[k] = L.X[ix0[k]]; g1[k] = L.A[ix1[k]]; }
+        else if constexpr (OP == JP_OP_PRIV_TMP) g0[k] = L.X[ix0[k]];
+        else { g0[k] = L.A[ix0[k]]; g1[k] = L.A[ix2[k]]; }
+      }
+    }
+    // ---------------- SE: values into the write log, write keys into the hash ----------------
+#pragma unroll
+    for (int k = 0; k < kTlsCtaIpt; k++) {
+      const int off = k * kTlsCtaThreads + tid;
+      if (off < span) {
+        if constexpr (OP == JP_OP_ADD_C) va[k] = op_add<DT>(g0[k], L.c0);
+        else if constexpr (OP == JP_OP_SAXPY) va[k] = op_add<DT>(op_mul<DT>(L.c0, g0[k]), g1[k]);
+        else if constexpr (OP == JP_OP_PRIV_TMP) { vt[k] = op_mul<DT>(L.c0, g0[k]); va[k] = op_add<DT>(vt[k], L.c1); }
+        else va[k] = op_mul<DT>(op_add<DT>(g0[k], g1[k]), L.c0);
+        if (P.hashA) slA[k] = hins(hk, hmin, hkey_of(ix1[k], 0), (uint32_t)off);
+        if constexpr (OP == JP_OP_PRIV_TMP) if (P.hashT) slT[k] = hins(hk, hmin, hkey_of(ix2[k], 1), (uint32_t)off);
+      }
+    }
+    TLS_SYNC();
     // ---------------- DC ----------------
     if (dc) {
       int myfv = INT32_MAX;
@@ -133,20 +198,22 @@ __global__ void __launch_bounds__(kTlsCtaThreads, 1) k_tls_cta(DLoop L, TlsArgs 
       for (int k = 0; k < kTlsCtaIpt; k++) {
         const int off = k * kTlsCtaThreads + tid;
         if (off < span && myfv == INT32_MAX) {
-          int h = hfind(hk, hkey_of(ra[k], 0));
+          // exposed reads of A: ADD_C/STENCIL2 A[r] (+ A[r2]); SAXPY Y[w]
+          const int32_t ra = OP == JP_OP_SAXPY ? ix1[k] : ix0[k];
+          int h = hfind(hk, hkey_of(ra, 0));
           bool v = h >= 0 && hmin[h] < (uint32_t)off;
           if constexpr (OP == JP_OP_STENCIL2) {
-            if (!v) { h = hfind(hk, hkey_of(rb[k], 0)); v = h >= 0 && hmin[h] < (uint32_t)off; }
+            if (!v) { h = hfind(hk, hkey_of(ix2[k], 0)); v = h >= 0 && hmin[h] < (uint32_t)off; }
           }
           if (v) myfv = off;
         }
       }
       myfv = __reduce_min_sync(0xffffffffu, myfv);
       if (lane == 0 && myfv != INT32_MAX) atomicMin(&s_fv[par], myfv);
-      __syncthreads();
+      TLS_SYNC();
     }
     const int fv = dc ? (s_fv[par] < span ? s_fv[par] : span) : span;
-    // ---------------- commit ----------------
+    // ---------------- commit [ws, ws+fv) ----------------
     if constexpr (WAW) {
 #pragma unroll
       for (int k = 0; k < kTlsCtaIpt; k++) {
@@ -156,18 +223,18 @@ __global__ void __launch_bounds__(kTlsCtaThreads, 1) k_tls_cta(DLoop L, TlsArgs 
           if constexpr (OP == JP_OP_PRIV_TMP) if (P.hashT) atomicMax(&hmax[slT[k]], (uint32_t)off + 1);
         }
       }
-      __syncthreads();
+      TLS_SYNC();
     }
 #pragma unroll
     for (int k = 0; k < kTlsCtaIpt; k++) {
       const int off = k * kTlsCtaThreads + tid;
       if (off < fv) {
-        if (!WAW || !P.hashA || hmax[slA[k]] == (uint32_t)off + 1) L.A[wa[k]] = va[k];
+        if (!WAW || !P.hashA || hmax[slA[k]] == (uint32_t)off + 1) L.A[ix1[k]] = va[k];
         if constexpr (OP == JP_OP_PRIV_TMP)
-          if (!WAW || !P.hashT || hmax[slT[k]] == (uint32_t)off + 1) L.T[wt[k]] = vt[k];
+          if (!WAW || !P.hashT || hmax[slT[k]] == (uint32_t)off + 1) L.T[ix2[k]] = vt[k];
       }
     }
-    if constexpr (WAW) __syncthreads();
+    if constexpr (WAW) TLS_SYNC();
     // clear the window's hash entries (no reader is left in this window)
 #pragma unroll
     for (int k = 0; k < kTlsCtaIpt; k++) {
@@ -182,7 +249,8 @@ __global__ void __launch_bounds__(kTlsCtaThreads, 1) k_tls_cta(DLoop L, TlsArgs 
     ws += fv;
     W = P.window > 0 ? P.window : next_window(L.n, P.prof_raw, fv, P.w_max);
     par ^= 1;
-    __syncthreads();   // commits visible to the next SE, hash clean
+    asm volatile("cp.async.wait_group 0;" ::: "memory");   // this window's prefetch has landed
+    TLS_SYNC();   // commits and prefetched indices visible to the next SE, hash clean
   }
   if (tid == 0) { stats[0] = committed; stats[1] = executed; stats[2] = windows; stats[3] = viol; }
 }
@@ -199,7 +267,7 @@ struct GridWs {
 };
 
 __device__ __forceinline__ void grid_sync(unsigned *bar) {
-  __syncthreads();
+  JP_CTA_SYNC();
   if (threadIdx.x == 0) {
     volatile unsigned *vgen = bar + 1;
     const unsigned g = *vgen;
@@ -213,7 +281,7 @@ __device__ __forceinline__ void grid_sync(unsigned *bar) {
     }
     __threadfence();
   }
-  __syncthreads();
+  JP_CTA_SYNC();
 }
 
 // body with L2-coherent (ld.global.cg) reads of the in/out array
@@ -324,7 +392,7 @@ template <int OP, int DT>
 static cudaError_t run_tls(const DLoop &d, const TlsPlan &p, TlsArgs a, void *ws, const Layout &lo, int64_t *stats,
                            cudaStream_t st) {
   if (p.path == 1) {
-    const size_t smem = 3 * kTlsHash * sizeof(uint32_t);
+    const size_t smem = 3 * kTlsHash * sizeof(uint32_t) + (size_t)n_streams<OP>() * kRing * sizeof(int32_t);
     if (p.waw) {
       cudaFuncSetAttribute(k_tls_cta<OP, DT, true>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
       k_tls_cta<OP, DT, true><<<1, kTlsCtaThreads, smem, st>>>(d, a, stats);

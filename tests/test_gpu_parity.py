@@ -460,3 +460,23 @@ def test_launch_count_and_version():
     torch.cuda.synchronize()
     assert jp.jp_launch_count() == n0 + 1
     assert "sm_100a" in jp.jp_version()
+
+
+@pytest.mark.parametrize("waw", [False, True])
+def test_tls_cta_repeatability(waw):
+    """The single-CTA window loop is timing sensitive (TLS
+    barrier): run the densest reduced config-3 loop 12 times per variant."""
+    wl = synth.config3(0.10, n=(1 << 17) + 11)
+    ref = to_oracle(wl)
+    _, A, _, stats = O.sim_tls(ref, 4096)
+    prof = None
+    for rep in range(12):
+        g = gpu(wl)
+        L = jp.Loop.from_workload(g)
+        ws = jp.workspace(L)
+        if not waw and prof is None:
+            prof = jp.jp_profile_density(L, ws)
+        got = jp.jp_run_tls(L, window=4096, w_max=4096, path=1, prof=None if waw else prof, ws=ws)
+        torch.cuda.synchronize()
+        assert got == stats, (rep, got, stats)
+        check_arrays(g, A, None)
