@@ -44,30 +44,45 @@ def peaks():
 
 
 class Clocks:
-    """nvidia-smi sampling during the timed region (B200_PROFILING.md clocks line)."""
+    """nvidia-smi sampling around the timed region (B200_PROFILING.md clocks line).
+    The sampler is started and primed before the timed region; samples taken
+    between the last one before the region and the first one after it count."""
     Q = ("clocks.sm,clocks.max.sm,clocks_event_reasons.active,clocks_event_reasons.hw_slowdown,"
          "clocks_event_reasons.hw_thermal_slowdown,clocks_event_reasons.sw_thermal_slowdown,"
          "clocks_event_reasons.sw_power_cap")
 
     def __init__(self, index: int):
         self.index, self.rows, self.proc = index, [], None
+        self.t0 = self.t1 = None
 
-    def __enter__(self):
+    def start(self):
         try:
             self.proc = subprocess.Popen(["nvidia-smi", "-i", str(self.index), f"--query-gpu={self.Q}",
-                                          "--format=csv,noheader,nounits", "-lms", "100"],
+                                          "--format=csv,noheader,nounits", "-lms", "50"],
                                          stdout=subprocess.PIPE, stderr=subprocess.DEVNULL, text=True)
             self.t = threading.Thread(target=self._read, daemon=True)
             self.t.start()
+            deadline = time.time() + 5.0
+            while not self.rows and time.time() < deadline:
+                time.sleep(0.01)
         except OSError:
             self.proc = None
         return self
 
     def _read(self):
         for line in self.proc.stdout:
-            self.rows.append([x.strip() for x in line.split(",")])
+            self.rows.append((time.time(), [x.strip() for x in line.split(",")]))
 
-    def __exit__(self, *a):
+    def mark_start(self):
+        self.t0 = time.time()
+
+    def mark_end(self):
+        self.t1 = time.time()
+        deadline = self.t1 + 1.0     # wait for the first sample after the region
+        while time.time() < deadline and not any(t > self.t1 for t, _ in self.rows):
+            time.sleep(0.01)
+
+    def stop(self):
         if self.proc:
             self.proc.terminate()
             try:
@@ -76,12 +91,18 @@ class Clocks:
                 self.proc.kill()
 
     def summary(self):
-        rows = [r for r in self.rows if len(r) >= 7 and r[0].isdigit()]
+        rows = [(t, r) for t, r in self.rows if len(r) >= 7 and r[0].isdigit()]
+        if self.t0 is not None and rows:
+            before = [t for t, _ in rows if t <= self.t0]
+            after = [t for t, _ in rows if t >= self.t1]
+            lo = before[-1] if before else self.t0
+            hi = after[0] if after else self.t1
+            rows = [(t, r) for t, r in rows if lo <= t <= hi]
         if not rows:
             return {"sm_mhz": None, "sm_max_mhz": None, "reasons": ["unsampled"], "samples": 0}
         names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
-        reasons = sorted({names[k] for r in rows for k in range(4) if r[3 + k].lower() == "active"})
-        return {"sm_mhz": statistics.median(int(r[0]) for r in rows), "sm_max_mhz": int(rows[0][1]),
+        reasons = sorted({names[k] for _, r in rows for k in range(4) if r[3 + k].lower() == "active"})
+        return {"sm_mhz": statistics.median(int(r[0]) for _, r in rows), "sm_max_mhz": int(rows[0][1][1]),
                 "reasons": reasons, "samples": len(rows)}
 
 
@@ -281,15 +302,18 @@ def run_jp(args):
     step = lambda: jp.jp_schedule(L, None, stream=st)  # noqa: E731  (static DOALL: no workspace needed)
     for _ in range(args.warmup):
         step()
+    clk = Clocks(local).start()
     barrier(world)
     n_launch0 = jp.jp_launch_count()
-    with Clocks(local) as clk:
-        t0 = torch.cuda.Event(enable_timing=True)
-        t1 = torch.cuda.Event(enable_timing=True)
-        t0.record(st)
-        per_step = time_steps(step, args.steps, st)
-        t1.record(st)
-        barrier(world)
+    clk.mark_start()
+    t0 = torch.cuda.Event(enable_timing=True)
+    t1 = torch.cuda.Event(enable_timing=True)
+    t0.record(st)
+    per_step = time_steps(step, args.steps, st)
+    t1.record(st)
+    barrier(world)
+    clk.mark_end()
+    clk.stop()
     launches = jp.jp_launch_count() - n_launch0
     total_ms = max_over_ranks(t0.elapsed_time(t1), world, dev)
     kernel_ms = max_over_ranks(statistics.mean(per_step), world, dev)
