@@ -56,14 +56,18 @@ typedef enum { JP_SCHED_SHARING = 0, JP_SCHED_STEALING = 1 } jp_scheme;
 
 typedef union { int32_t i; float f; } jp_scalar;
 
-/* Loop descriptor.  Index arrays are int32 [n]; NULL means identity (index i).
- * Element arrays are 4-byte int32 or fp32 per `dtype`; A, X, T must not alias
- * each other (reading A14).  Global iteration id of local iteration i is
- * iter_base + i (used by stamps and keys so that chunks/ranks compose); all
- * global ids must be < 2^31 - 1.                                               */
+/* Loop descriptor.  Index arrays are int32 [n]; NULL means identity: local
+ * iteration i accesses element ident_off + i.  Element arrays are 4-byte int32
+ * or fp32 per `dtype`; A, X, T must not alias each other (reading A14).  Global
+ * iteration id of local iteration i is iter_base + i (used by stamps and keys
+ * so that chunks/ranks compose); all global ids must be < 2^31 - 1.  A whole
+ * loop has iter_base = ident_off = 0; a rank's range [b, e) of a loop over
+ * full-size replicas has n = e-b, iter_base = ident_off = b and index arrays
+ * offset by b; a range over sharded identity-only arrays keeps ident_off = 0. */
 typedef struct {
   int64_t n;                    /* trip count, 0 <= n, iter_base + n <= 2^31-2        */
   int64_t iter_base;            /* global id of local iteration 0                     */
+  int64_t ident_off;            /* element index of local iteration 0 under identity  */
   int32_t op;                   /* jp_op                                              */
   int32_t dtype;                /* jp_dtype                                           */
   const int32_t *r, *r2, *w, *s;

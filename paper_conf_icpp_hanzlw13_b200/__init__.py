@@ -50,7 +50,7 @@ class Loop:
     not copied: the kernels update A (and T) in place."""
 
     def __init__(self, op, dtype, n, A, r=None, r2=None, w=None, s=None, X=None, T=None, c0=0, c1=0,
-                 iter_base=0):
+                 iter_base=0, ident_off=0):
         el = _EL[dtype]
         for name, t in (("A", A), ("X", X), ("T", T)):
             if t is not None and (t.dtype != el or not t.is_contiguous()):
@@ -61,11 +61,13 @@ class Loop:
         self.tensors = dict(A=A, r=r, r2=r2, w=w, s=s, X=X, T=T)
         self.op, self.dtype, self.n = int(op), int(dtype), int(n)
         c = _abi.jp_loop()
-        c.n, c.iter_base, c.op, c.dtype = self.n, int(iter_base), self.op, self.dtype
+        c.n, c.iter_base, c.ident_off, c.op, c.dtype = self.n, int(iter_base), int(ident_off), self.op, self.dtype
+        self.iter_base, self.ident_off = int(iter_base), int(ident_off)
         c.r, c.r2, c.w, c.s = _ptr(r), _ptr(r2), _ptr(w), _ptr(s)
         c.A, c.len_A = _ptr(A), (0 if A is None else A.numel())
         c.X, c.len_X = _ptr(X), (0 if X is None else X.numel())
         c.T, c.len_T = _ptr(T), (0 if T is None else T.numel())
+        self._c0, self._c1 = c0, c1
         for slot, v in (("c0", c0), ("c1", c1)):
             sc = _abi.jp_scalar()
             if dtype == JP_F32:
@@ -76,9 +78,18 @@ class Loop:
         self.c = c
 
     @classmethod
-    def from_workload(cls, wl, iter_base: int = 0):
+    def from_workload(cls, wl, iter_base: int = 0, ident_off: int = 0):
         return cls(wl.op, wl.dtype, wl.n, wl.A, r=wl.r, r2=wl.r2, w=wl.w, s=wl.s, X=wl.X, T=wl.T, c0=wl.c0,
-                   c1=wl.c1, iter_base=iter_base)
+                   c1=wl.c1, iter_base=iter_base, ident_off=ident_off)
+
+    def range(self, b: int, e: int) -> "Loop":
+        """This loop's iterations [b, e) as a rank-local loop over the same
+        (full-size) arrays: iter_base = ident_off = b, index arrays offset."""
+        t = self.tensors
+        sl = lambda x: None if x is None else x[b:e]  # noqa: E731
+        return Loop(self.op, self.dtype, e - b, t["A"], r=sl(t["r"]), r2=sl(t["r2"]), w=sl(t["w"]), s=sl(t["s"]),
+                    X=t["X"], T=t["T"], c0=self._c0, c1=self._c1, iter_base=self.iter_base + b,
+                    ident_off=self.ident_off + b)
 
     @property
     def ref(self):

@@ -34,7 +34,7 @@ class jp_scalar(C.Union):
 
 class jp_loop(C.Structure):
     _fields_ = [
-        ("n", C.c_int64), ("iter_base", C.c_int64), ("op", C.c_int32), ("dtype", C.c_int32),
+        ("n", C.c_int64), ("iter_base", C.c_int64), ("ident_off", C.c_int64), ("op", C.c_int32), ("dtype", C.c_int32),
         ("r", C.c_void_p), ("r2", C.c_void_p), ("w", C.c_void_p), ("s", C.c_void_p),
         ("A", C.c_void_p), ("len_A", C.c_int64),
         ("X", C.c_void_p), ("len_X", C.c_int64),

@@ -77,7 +77,7 @@ Job make_job(const jp_loop *L) {
   DLoop &d = j.d;
   d.n = L->n;
   d.base = L->iter_base;
-  d.ioff = 0;
+  d.ioff = L->ident_off;
   d.r = ur ? L->r : nullptr;
   d.r2 = ur2 ? L->r2 : nullptr;
   d.w = uw ? L->w : nullptr;
@@ -161,8 +161,8 @@ static jp_status check_loop(const jp_loop *L) {
   if (!L) return fail(JP_ERR_ARG, "loop descriptor is NULL");
   if (L->op < JP_OP_ADD_C || L->op > JP_OP_STENCIL2) return fail(JP_ERR_UNSUPPORTED, "opcode %d is not templated", L->op);
   if (L->dtype != JP_I32 && L->dtype != JP_F32) return fail(JP_ERR_UNSUPPORTED, "dtype %d is not templated", L->dtype);
-  if (L->n < 0 || L->iter_base < 0 || L->iter_base + L->n > 2147483646LL)
-    return fail(JP_ERR_ARG, "need 0 <= n, 0 <= iter_base, iter_base + n <= 2^31-2 (n=%lld base=%lld)",
+  if (L->n < 0 || L->iter_base < 0 || L->iter_base + L->n > 2147483646LL || L->ident_off < 0)
+    return fail(JP_ERR_ARG, "need 0 <= n, 0 <= iter_base, 0 <= ident_off, iter_base + n <= 2^31-2 (n=%lld base=%lld)",
                 (long long)L->n, (long long)L->iter_base);
   const int64_t lmax = 2147483647LL;
   if (L->len_A < 0 || L->len_X < 0 || L->len_T < 0 || L->len_A > lmax || L->len_X > lmax || L->len_T > lmax)
@@ -174,8 +174,9 @@ static jp_status check_loop(const jp_loop *L) {
   if (L->op == JP_OP_PRIV_TMP && !L->T) return fail(JP_ERR_ARG, "T is NULL");
   // identity accesses must stay inside their arrays (reading A13)
   auto idn = [&](const int32_t *p, int64_t len, const char *what) -> jp_status {
-    if (!p && L->n > len) return fail(JP_ERR_INDEX, "identity index of %s exceeds its length (%lld > %lld)", what,
-                                      (long long)L->n, (long long)len);
+    if (!p && L->ident_off + L->n > len)
+      return fail(JP_ERR_INDEX, "identity index of %s exceeds its length (%lld > %lld)", what,
+                  (long long)(L->ident_off + L->n), (long long)len);
     return JP_OK;
   };
   jp_status s = JP_OK;

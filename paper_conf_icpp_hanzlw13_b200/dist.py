@@ -1,0 +1,140 @@
+"""Multi-GPU driver: the paper's task-sharing and task-stealing schemes
+(Sec. V) across the ranks of one node, one process per GPU.
+
+The C library never calls NCCL (include/jp.h): this module issues the
+collectives through ``torch.distributed`` between the split entry points of
+libjp.so and lets the kernels consume the results.  Collectives used
+(SURVEY.md Sec.2c):
+
+  C1  all_reduce MAX int32  over the first-writer / first-reader tables of the
+      partitioned profile (entries are INT32_MAX - gid, empty -1);
+  C3  all_reduce SUM int64  over the per-rank raw/war/waw counts;
+  C4  all_reduce MAX int64  over the packed last-writer keys (gid+1)<<32|bits
+      of the privatized / partitioned writes;
+  bcast                      of the in/out array after a TLS run (TLS windows
+      stay ordered on one GPU: "replicas only", north_star).
+
+Iteration ranges come from ``jp_plan_sharing`` (boundary formula)
+and ``jp_plan_stealing`` (Alg. 1).  Every compute step is a
+libjp.so kernel; ``engine`` exists only so that the CPU tests can drive the
+collective logic with gloo and a test double (there is no CPU path here).
+"""
+from __future__ import annotations
+
+import torch
+import torch.distributed as dist
+
+from . import _abi
+
+
+def _engine(engine):
+    if engine is not None:
+        return engine
+    import paper_conf_icpp_hanzlw13_b200 as jp
+    return jp
+
+
+def world_rank(group=None) -> tuple[int, int]:
+    if dist.is_available() and dist.is_initialized():
+        return dist.get_world_size(group), dist.get_rank(group)
+    return 1, 0
+
+
+def sharing_ranges(n: int, world: int, weights=None, engine=None):
+    """Task-sharing plan: rank k gets [floor(n*S_k), floor(n*S_{k+1}))."""
+    return _engine(engine).jp_plan_sharing(n, world, weights)
+
+
+def _region(ws: torch.Tensor, loop, name: str, dtype, engine=None):
+    off, nb = _engine(engine).jp_ws_region(loop, name)
+    if nb == 0:
+        return None
+    return ws[off:off + nb].view(dtype)
+
+
+def profile_partitioned(loop, ws, group=None, engine=None) -> dict:
+    """Profile of the whole loop from rank-local ranges (iter_base = global id of
+    the rank's first iteration): stamp locally, C1, classify locally, C3.  The
+    result equals the single-GPU profile exactly (tested)."""
+    jp = _engine(engine)
+    world, _ = world_rank(group)
+    jp.jp_profile_stamp(loop, ws)
+    if world > 1:
+        for name in ("minW_A", "minR_A", "minW_T", "minR_T"):
+            t = _region(ws, loop, name, torch.int32, jp)
+            if t is not None:
+                dist.all_reduce(t, op=dist.ReduceOp.MAX, group=group)
+    p = jp.jp_profile_classify(loop, ws)
+    if world > 1:
+        dev = ws.device
+        c = torch.tensor([p["n"], p["raw_iters"], p["war_iters"], p["waw_iters"]], dtype=torch.int64, device=dev)
+        dist.all_reduce(c, group=group)
+        f = torch.tensor([p["first_raw_iter"] if p["first_raw_iter"] >= 0 else (1 << 62)], dtype=torch.int64,
+                         device=dev)
+        dist.all_reduce(f, op=dist.ReduceOp.MIN, group=group)
+        n, raw, war, waw = (int(x) for x in c.tolist())
+        fr = int(f.item())
+        p = {"n": n, "raw_iters": raw, "war_iters": war, "waw_iters": waw,
+             "first_raw_iter": -1 if fr >= (1 << 62) else fr,
+             "d_raw": raw / n if n else 0.0, "d_war": war / n if n else 0.0, "d_waw": waw / n if n else 0.0}
+    return p
+
+
+def privatized_partitioned(loop, ws, prof, group=None, engine=None):
+    """PE(V) over rank-local ranges: keys locally, C4 (MAX over packed keys), then
+    every rank applies the merged keys -- each rank ends with the sequential
+    result in its replica of the keyed arrays; identity-indexed outputs stay
+    sharded (each rank holds its own range)."""
+    jp = _engine(engine)
+    world, _ = world_rank(group)
+    jp.jp_priv_stream(loop, prof, ws, clear_keys=True)
+    if world > 1:
+        for name in ("keys_A", "keys_T"):
+            t = _region(ws, loop, name, torch.int64, jp)
+            if t is not None:
+                dist.all_reduce(t, op=dist.ReduceOp.MAX, group=group)
+    jp.jp_priv_finalize(loop, ws)
+
+
+def schedule_partitioned(loop, ws, group=None, tau_high: float = 0.25, tls_window: int = 0, tls_w_max: int = 4096,
+                         full_loop=None, engine=None) -> dict:
+    """Task sharing of one loop across the ranks (P:L342-358 generalised to k
+    devices).  ``loop`` is this rank's range (iter_base = its first global id,
+    index arrays offset, element arrays shared-address replicas).
+
+      * all index arrays NULL: determined DOALL, each rank runs its shard, no
+        collective (outputs stay sharded);
+      * else partitioned profile (C1+C3), Fig. 2(b) mode, then
+        DOALL / PRIVATIZED: privatized kernels + C4 merge (a DOALL loop is the
+        dependence-free special case of PE(V));
+        TLS / SEQ_RECOMMENDED: rank 0 runs the windows over ``full_loop`` and
+        broadcasts the in/out arrays (replicas only).
+    """
+    jp = _engine(engine)
+    world, rank = world_rank(group)
+    if loop.tensors["r"] is None and loop.tensors["w"] is None and loop.tensors["r2"] is None \
+            and loop.tensors["s"] is None:
+        res = jp.jp_schedule(loop, ws)
+        res["scheme"] = "sharing"
+        return res
+    prof = profile_partitioned(loop, ws, group, jp)
+    mode = jp.jp_select_mode(loop, prof, tau_high)
+    res = {"mode": mode, "mode_name": _abi.MODE_NAMES[mode], "profiled": 1, "prof": prof, "scheme": "sharing"}
+    if mode in (_abi.JP_MODE_DOALL, _abi.JP_MODE_PRIVATIZED):
+        privatized_partitioned(loop, ws, prof, group, jp)
+    else:
+        if full_loop is None:
+            raise ValueError("TLS needs the whole loop on rank 0 (full_loop)")
+        if rank == 0:
+            res["tls"] = jp.jp_run_tls(full_loop, window=tls_window, w_max=tls_w_max, prof=prof, ws=ws)
+        if world > 1:
+            for name in ("A", "T"):
+                t = full_loop.tensors[name]
+                if t is not None:
+                    dist.broadcast(t, src=0, group=group)
+    return res
+
+
+def stealing_plan(tasks, world: int, chunk_iters: int, speed=None, speed_tls: float = 0.05, engine=None):
+    """Alg. 1 as a deterministic plan: [(start, end, mode, owner)] and #stolen."""
+    return _engine(engine).jp_plan_stealing(tasks, world, chunk_iters, speed, speed_tls)

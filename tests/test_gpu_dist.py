@@ -1,0 +1,77 @@
+"""Multi-process partitioned runs with the REAL kernels: world_size 2 ranks share
+cuda:0 over the gloo backend (the only GPU a test box has), each rank running
+its task-sharing range through libjp.so and dist.py's collectives (C1, C3, C4,
+TLS broadcast).  The NCCL/NVLink path uses the same code with backend "nccl"."""
+import os
+import socket
+import sys
+
+import pytest
+import torch
+import torch.distributed as dist
+import torch.multiprocessing as mp
+
+pytestmark = pytest.mark.gpu
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+
+
+def _port():
+    s = socket.socket()
+    s.bind(("127.0.0.1", 0))
+    p = s.getsockname()[1]
+    s.close()
+    return p
+
+
+def _worker(rank, world, port, case, q):
+    sys.path[:0] = [ROOT, os.path.join(ROOT, "tests")]
+    os.environ.update(MASTER_ADDR="127.0.0.1", MASTER_PORT=str(port))
+    dist.init_process_group("gloo", rank=rank, world_size=world)
+    try:
+        import oracle as O
+        import paper_conf_icpp_hanzlw13_b200 as jp
+        from paper_conf_icpp_hanzlw13_b200 import dist as jd
+        import synth
+        from helpers import to_oracle
+        dev = torch.device("cuda:0")
+        wl = {"c1_0": lambda: synth.config1(0.0), "c1_5": lambda: synth.config1(0.05),
+              "c4": lambda: synth.config4(n=(1 << 18) + 5), "c3": lambda: synth.config3(0.01, n=1 << 16),
+              "c5tail": lambda: synth.config5(n=1 << 14)}[case]()
+        ref = to_oracle(wl)
+        _, A_exp, T_exp = O.run_seq(ref)
+        g = wl.to(dev)
+        full = jp.Loop.from_workload(g)
+        b, e = jd.sharing_ranges(wl.n, world)[rank]
+        loop = full.range(b, e)
+        ws = jp.workspace(loop)
+        res = jd.schedule_partitioned(loop, ws, full_loop=full)
+        torch.cuda.synchronize()
+        if wl.op == O.OP_PRIV_TMP:
+            ok = g.A.cpu().numpy()[b:e].tobytes() == A_exp[b:e].tobytes() and \
+                g.T.cpu().numpy().tobytes() == T_exp.tobytes()
+        else:
+            ok = g.A.cpu().numpy().tobytes() == A_exp.tobytes()
+        p = O.profile(ref)
+        ok &= (res["prof"]["raw_iters"], res["prof"]["war_iters"], res["prof"]["waw_iters"]) == \
+            (p["raw_iters"], p["war_iters"], p["waw_iters"])
+        q.put((rank, bool(ok), res["mode_name"]))
+    except Exception as ex:  # pragma: no cover
+        q.put((rank, False, repr(ex)))
+    finally:
+        dist.destroy_process_group()
+
+
+@pytest.mark.parametrize("case,mode", [("c1_0", "DOALL"), ("c1_5", "TLS"), ("c4", "PRIVATIZED"), ("c3", "TLS"),
+                                       ("c5tail", "TLS")])
+def test_two_ranks_one_gpu(case, mode):
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    port = _port()
+    ps = [ctx.Process(target=_worker, args=(r, 2, port, case, q)) for r in range(2)]
+    for p in ps:
+        p.start()
+    out = sorted(q.get(timeout=600) for _ in range(2))
+    for p in ps:
+        p.join(timeout=120)
+    assert [o[1] for o in out] == [True, True], out
+    assert all(o[2] == mode for o in out), out
