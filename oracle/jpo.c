@@ -198,6 +198,29 @@ int jpo_pairs(const jpo_loop *L, jpo_profile *out, uint8_t *flags) {
   return JPO_OK;
 }
 
+/* RAW sources (profile-guided mode B): src[j] = 1 iff
+ * some write of j is an exposed read of a LATER iteration, i.e. j is the
+ * earlier end of a RAW pair (W(j) ∩ R_exp(i) != {} for some i > j, reading
+ * A1's pair relation).  Single backward pass: before recording i's exposed
+ * reads, its writes are checked against the addresses read by iterations > i.
+ * Only such writes can make an in-window RAW violation (reading A7).       */
+int jpo_raw_sources(const jpo_loop *L, uint8_t *src) {
+  if (!op_valid(L) || !src) return JPO_ERR_ARG;
+  int e = check_indices(L); if (e) return e;
+  int64_t len[3] = {L->len_A, L->len_X, L->len_T};
+  uint8_t *read_after[3];
+  for (int k = 0; k < 3; k++) read_after[k] = (uint8_t *)calloc(len[k] > 0 ? len[k] : 1, 1);
+  for (int64_t i = L->n - 1; i >= 0; i--) {
+    accs_t s; accesses(L, i, &s);
+    int f = 0;
+    for (int k = 0; k < s.nwr; k++) if (read_after[s.wr[k].arr][s.wr[k].a]) f = 1;
+    src[i] = (uint8_t)f;
+    for (int k = 0; k < s.nrexp; k++) read_after[s.rexp[k].arr][s.rexp[k].a] = 1;
+  }
+  for (int k = 0; k < 3; k++) free(read_after[k]);
+  return JPO_OK;
+}
+
 /* ---------------------------------------------------------------------------
  * GPU-TLS as a definition (P:L314-333 SE/DC/commit/recovery; P:L367-375 mode
  * B restarts "from the violating warp"; readings A6, A7, A8):

@@ -62,6 +62,8 @@ int jpo_run_order(const jpo_loop *L, const int64_t *perm);
 int jpo_profile_run(const jpo_loop *L, jpo_profile *out, uint8_t *flags);
 /* O(n^2) enumeration of all ordered pairs (item 3); same flags + pair counts. */
 int jpo_pairs(const jpo_loop *L, jpo_profile *out, uint8_t *flags);
+/* RAW sources: src[j] = 1 iff a write of j is exposed-read by some i > j. */
+int jpo_raw_sources(const jpo_loop *L, uint8_t *src);
 /* Windowed TLS as a definition (item 4).  window > 0: fixed W.  window == 0:
  * adaptive policy of reading A8 with cap w_max; prof_raw_iters < 0 means "no
  * profile known".  Modifies the arrays (must end equal to jpo_run_seq).      */

@@ -61,6 +61,7 @@ def _load():
             lib.jpo_run_order.argtypes = [P(_Loop), C.c_void_p]
             lib.jpo_profile_run.argtypes = [P(_Loop), P(_Profile), C.c_void_p]
             lib.jpo_pairs.argtypes = [P(_Loop), P(_Profile), C.c_void_p]
+            lib.jpo_raw_sources.argtypes = [P(_Loop), C.c_void_p]
             lib.jpo_sim_tls.argtypes = [P(_Loop), C.c_int64, C.c_int64, C.c_int64, P(_TlsStats)]
             lib.jpo_tls_next_window.argtypes = [C.c_int64] * 4
             lib.jpo_tls_next_window.restype = C.c_int64
@@ -139,6 +140,15 @@ def profile(loop: Loop) -> dict:
 def pairs(loop: Loop) -> dict:
     """O(n^2) pair enumeration (brute force)."""
     return _prof(_load().jpo_pairs, loop)
+
+
+def raw_sources(loop: Loop) -> np.ndarray:
+    """src[j] = 1 iff a write of j is an exposed read of a later iteration."""
+    src = np.zeros(max(loop.n, 1), dtype=np.uint8)
+    st = _load().jpo_raw_sources(C.byref(loop._c()), src.ctypes.data)
+    if st != OK:
+        raise ValueError(f"jpo_raw_sources: status {st}")
+    return src[: loop.n]
 
 
 def sim_tls(loop: Loop, window: int, w_max: int = 65536, prof_raw_iters: int = -1):

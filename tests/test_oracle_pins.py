@@ -53,6 +53,12 @@ def brute_profile(op, n, r=None, r2=None, w=None, s=None):
     return raw, war, waw, flags
 
 
+def brute_sources(op, n, r=None, r2=None, w=None, s=None):
+    """RAW sources over all ordered pairs: j with W(j) ∩ R_exp(i) != {} for an i > j."""
+    sets = [acc_sets(op, i, r, r2, w, s) for i in range(n)]
+    return [int(any(set(sets[j][2]) & set(sets[i][0]) for i in range(j + 1, n))) for j in range(n)]
+
+
 def brute_tls_stats(op, n, W, r=None, r2=None, w=None, s=None):
     """Reading A6: fv = first i in the window with an earlier in-window writer of
     one of its exposed reads (O(W^2)); prefix commit; restart at fv."""
@@ -153,6 +159,7 @@ def test_profile_exhaustive_vs_bruteforce():
         b = brute_profile(O.OP_ADD_C, n, r=r, w=w)
         assert (p["raw_iters"], p["war_iters"], p["waw_iters"]) == b[:3]
         assert p["flags"].tolist() == b[3]
+        assert O.raw_sources(L).tolist() == brute_sources(O.OP_ADD_C, n, r=r, w=w)
         if p["raw_iters"] == 0:
             seen_zero += 1
     assert seen_zero == 1728  # the count the survey's brute force found
@@ -185,6 +192,7 @@ def test_profile_random_all_ops_vs_bruteforce(seed):
     b = brute_profile(op, n, r=r, r2=r2, w=w, s=s)
     assert (p["raw_iters"], p["war_iters"], p["waw_iters"]) == b[:3]
     assert p["flags"].tolist() == b[3] == q["flags"].tolist()
+    assert O.raw_sources(L).tolist() == brute_sources(op, n, r=r, r2=r2, w=w, s=s)
     # TLS: arrays equal the sequential run, stats equal the O(W^2) definition
     for W in (1, 2, 3, 5, 16):
         st, A, T, stats = O.sim_tls(L, W)
@@ -213,6 +221,22 @@ def test_tls_exhaustive_invariants():
                 assert st["violations"] == 0 and st["windows"] == -(-n // W)
         if raw == 0:
             assert O.sim_priv(L)[1].tolist() == seq.tolist()
+
+
+@pytest.mark.parametrize("n", [1, 2, 9, 500])
+def test_raw_sources_closed_forms(n):
+    """Closed forms: the prefix chain's sources are every iteration but the last;
+    a permutation self-update has none; Gauss-Seidel's are all but the last."""
+    ar = np.arange(n, dtype=np.int32)
+    A0 = np.zeros(n, dtype=np.int32)
+    pc = O.Loop(O.OP_ADD_C, O.I32, n, A0, r=np.maximum(ar - 1, 0), w=ar, c0=1)
+    # j writes j and iteration j+1 reads it; the last write is never read later
+    assert O.raw_sources(pc).tolist() == [1] * (n - 1) + [0]
+    perm = np.random.default_rng(n).permutation(n).astype(np.int32)
+    assert O.raw_sources(O.Loop(O.OP_ADD_C, O.I32, n, A0, r=perm, w=perm, c0=1)).tolist() == [0] * n
+    gs = O.Loop(O.OP_STENCIL2, O.I32, n, A0, r=np.maximum(ar - 1, 0), r2=np.minimum(ar + 1, n - 1), w=ar, c0=1)
+    # j is read later by j+1 (through r = j); the last iteration's write is never read later
+    assert O.raw_sources(gs).tolist() == [1] * (n - 1) + [0]
 
 
 def test_priv_counterexample_prefix_chain():
