@@ -93,9 +93,19 @@ typedef struct { int64_t committed, executed, windows, violations; } jp_tls_stat
 /* TLS window policy (reading A8).  window > 0: fixed W.  window == 0: adaptive,
  * W0 = clamp(pow2ceil(ceil(4n/raw)),32,w_max) with a profile (w_max if raw == 0,
  * 4096 without profile), then W <- clamp(pow2ceil(2*max(c,16)), 32, w_max)
- * after a window that committed c iterations.  path: 0 auto, 1 single-CTA
- * shared-memory path (W <= 4096), 2 cooperative all-SM path (HBM stamps).     */
-typedef struct { int64_t window; int64_t w_max; int32_t path; int32_t reserved; } jp_tls_cfg;
+ * after a window that committed c iterations.  path: 0 auto (3 when the
+ * window fits a 16-CTA cluster, else 2), 1 single-CTA shared-memory hash path
+ * (W <= 4096), 2 cooperative all-SM path (HBM stamps, software grid barrier),
+ * 3 one thread-block cluster of `cluster` CTAs (HBM stamps, cluster barriers,
+ * W <= 32*(144*cluster - 1)).  cluster: 1..16, 0 = auto (smallest power of two
+ * >= 4 that holds the window); ignored by paths 1 and 2.                       */
+typedef struct {
+  int64_t window; int64_t w_max; int32_t path; int32_t cluster;
+  int32_t guided;   /* 1: use the guide bitmaps (region 13) that jp_tls_guide wrote for
+                       this loop on this workspace; needs a profile with waw_iters == 0
+                       (JP_ERR_ARG otherwise).  Same windows, stats and arrays.   */
+  int32_t reserved;
+} jp_tls_cfg;
 
 typedef struct {
   int32_t scheme;               /* jp_scheme                                          */
@@ -124,11 +134,13 @@ typedef struct {
  * region any of the requested uses (JP_WS_* bits) needs, so a buffer sized for
  * more uses serves every smaller one.  Functions return JP_ERR_WORKSPACE when
  * ws_bytes is too small for what they touch.                                   */
-enum { JP_WS_PROFILE = 1, JP_WS_PRIV = 2, JP_WS_TLS = 4, JP_WS_SCHED = 8, JP_WS_ALL = 15 };
+enum { JP_WS_PROFILE = 1, JP_WS_PRIV = 2, JP_WS_TLS = 4, JP_WS_SCHED = 8, JP_WS_GUIDE = 16, JP_WS_ALL = 31 };
 size_t jp_workspace_bytes(const jp_loop *L /* host */, int32_t uses);
 /* region ids: 0 header, 1 minW(A) int32, 2 minR(A) int32, 3 minW(T), 4 minR(T),
  * 5 keys(A) int64, 6 keys(T) int64, 7 tls stamps(A) u64, 8 tls commit(A) u64,
- * 9 (reserved), 10 tls commit(T) u64, 11 scheduler scratch.  Stamp tables hold
+ * 9 (reserved), 10 tls commit(T) u64, 11 scheduler scratch, 12 latest exposed
+ * reader maxRx(A) int32 (gid, empty -1), 13 TLS guide bitmaps u32 [2][ceil(n/32)]
+ * (raw words, then RAW-source words; see jp_tls_guide).  Stamp tables hold
  * INT32_MAX - gid (empty = -1) so that an all_reduce MAX over int32 yields the
  * global first writer/reader; keys hold (gid+1)<<32 | bits32(value) (empty = 0)
  * so that an all_reduce MAX over int64 yields the global last writer.  bytes = 0
@@ -199,6 +211,17 @@ jp_status jp_priv_finalize(const jp_loop *L, void *ws, size_t ws_bytes, jp_strea
  * window loop runs inside one persistent kernel.  stats (host, nullable): if
  * non-NULL the call syncs.  prof (host, nullable) feeds the adaptive policy and
  * lets the commit skip WAW resolution when waw_iters == 0.                   */
+/* TLS guide (profile-guided mode B; P:L369-375 uses the
+ * profiled density to steer mode B).  From the first-writer table of a
+ * jp_profile_stamp on the SAME workspace and loop, fills region 13 with
+ *   raw_i = an exposed read of i was written by an earlier iteration, and
+ *   src_j = the write of j is an exposed read of some later iteration
+ * (a maxRx pass over the exposed reads, region 12).  An in-window RAW
+ * violation (reading A7) needs a raw reader and a source writer, so a guided
+ * TLS run stamps only sources and checks only raw readers and finds exactly
+ * the same first violators.  Needs JP_WS_PROFILE | JP_WS_GUIDE.  No sync.
+ * Loops whose A is not reached through an index have no guide (no-op).     */
+jp_status jp_tls_guide(const jp_loop *L, void *ws, size_t ws_bytes, jp_stream_t st);
 jp_status jp_run_tls(const jp_loop *L, const jp_tls_cfg *cfg /* host */, const jp_profile *prof,
                      void *ws, size_t ws_bytes, jp_tls_stats *stats, jp_stream_t st);
 

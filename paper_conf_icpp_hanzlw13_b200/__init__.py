@@ -16,14 +16,14 @@ from . import _abi
 from ._abi import (  # noqa: F401
     JP_I32, JP_F32, JP_OP_ADD_C, JP_OP_SAXPY, JP_OP_PRIV_TMP, JP_OP_STENCIL2,
     JP_MODE_DOALL, JP_MODE_PRIVATIZED, JP_MODE_TLS, JP_MODE_SEQ_RECOMMENDED, MODE_NAMES,
-    JP_SCHED_SHARING, JP_SCHED_STEALING, JP_WS_PROFILE, JP_WS_PRIV, JP_WS_TLS, JP_WS_SCHED, JP_WS_ALL,
+    JP_SCHED_SHARING, JP_SCHED_STEALING, JP_WS_PROFILE, JP_WS_PRIV, JP_WS_TLS, JP_WS_SCHED, JP_WS_GUIDE, JP_WS_ALL,
     REGIONS, JPError, check, lib,
 )
 
 __all__ = [
     "Loop", "workspace", "jp_workspace_bytes", "jp_ws_region", "jp_validate", "jp_profile_stamp",
     "jp_profile_classify", "jp_profile_density", "jp_select_mode", "jp_run_doall", "jp_run_privatized",
-    "jp_priv_stream", "jp_priv_finalize", "jp_run_tls", "jp_schedule", "jp_stage_bytes", "jp_schedule_host",
+    "jp_priv_stream", "jp_priv_finalize", "jp_tls_guide", "jp_run_tls", "jp_schedule", "jp_stage_bytes", "jp_schedule_host",
     "jp_plan_sharing", "jp_plan_stealing", "jp_merge_apply", "jp_last_error", "jp_version", "jp_launch_count",
 ]
 
@@ -193,8 +193,15 @@ def jp_priv_finalize(loop: Loop, ws, stream=None):
     check(lib().jp_priv_finalize(loop.ref, p, nb, _stream(stream)))
 
 
-def jp_run_tls(loop: Loop, window=0, w_max=65536, path=0, prof=None, ws=None, stats=True, stream=None):
-    cfg = _abi.jp_tls_cfg(int(window), int(w_max), int(path), 0)
+def jp_tls_guide(loop: Loop, ws: torch.Tensor, stream=None) -> None:
+    """Guide bitmaps (region 13) from a profile already run on `ws` (jp.h)."""
+    p, nb = _ws(ws)
+    check(lib().jp_tls_guide(loop.ref, p, nb, _stream(stream)))
+
+
+def jp_run_tls(loop: Loop, window=0, w_max=65536, path=0, prof=None, ws=None, stats=True, stream=None, cluster=0,
+               guided=False):
+    cfg = _abi.jp_tls_cfg(int(window), int(w_max), int(path), int(cluster), int(bool(guided)), 0)
     st = _abi.jp_tls_stats()
     p, nb = _ws(ws)
     check(lib().jp_run_tls(loop.ref, C.byref(cfg), _pref(prof), p, nb, C.byref(st) if stats else None,

@@ -23,9 +23,9 @@ JP_OP_ADD_C, JP_OP_SAXPY, JP_OP_PRIV_TMP, JP_OP_STENCIL2 = 0, 1, 2, 3
 JP_MODE_DOALL, JP_MODE_PRIVATIZED, JP_MODE_TLS, JP_MODE_SEQ_RECOMMENDED = 0, 1, 2, 3
 MODE_NAMES = {0: "DOALL", 1: "PRIVATIZED", 2: "TLS", 3: "SEQ_RECOMMENDED"}
 JP_SCHED_SHARING, JP_SCHED_STEALING = 0, 1
-JP_WS_PROFILE, JP_WS_PRIV, JP_WS_TLS, JP_WS_SCHED, JP_WS_ALL = 1, 2, 4, 8, 15
+JP_WS_PROFILE, JP_WS_PRIV, JP_WS_TLS, JP_WS_SCHED, JP_WS_GUIDE, JP_WS_ALL = 1, 2, 4, 8, 16, 31
 REGIONS = {"header": 0, "minW_A": 1, "minR_A": 2, "minW_T": 3, "minR_T": 4, "keys_A": 5, "keys_T": 6,
-           "tls_S_A": 7, "tls_C_A": 8, "tls_C_T": 10, "sched": 11}
+           "tls_S_A": 7, "tls_C_A": 8, "tls_C_T": 10, "sched": 11, "maxRx_A": 12, "guide": 13}
 
 
 class jp_scalar(C.Union):
@@ -55,7 +55,8 @@ class jp_tls_stats(C.Structure):
 
 
 class jp_tls_cfg(C.Structure):
-    _fields_ = [("window", C.c_int64), ("w_max", C.c_int64), ("path", C.c_int32), ("reserved", C.c_int32)]
+    _fields_ = [("window", C.c_int64), ("w_max", C.c_int64), ("path", C.c_int32), ("cluster", C.c_int32),
+                ("guided", C.c_int32), ("reserved", C.c_int32)]
 
 
 class jp_sched_cfg(C.Structure):
@@ -82,6 +83,7 @@ SIGNATURES = [
     ("jp_run_privatized", _I32, [_P(jp_loop), _P(jp_profile), _V, _SZ, _V]),
     ("jp_priv_stream", _I32, [_P(jp_loop), _P(jp_profile), _V, _SZ, _I32, _V]),
     ("jp_priv_finalize", _I32, [_P(jp_loop), _V, _SZ, _V]),
+    ("jp_tls_guide", _I32, [_P(jp_loop), _V, _SZ, _V]),
     ("jp_run_tls", _I32, [_P(jp_loop), _P(jp_tls_cfg), _P(jp_profile), _V, _SZ, _P(jp_tls_stats), _V]),
     ("jp_schedule", _I32, [_P(jp_loop), _P(jp_sched_cfg), _V, _SZ, _P(jp_sched_result), _V]),
     ("jp_stage_bytes", _SZ, [_P(jp_loop)]),

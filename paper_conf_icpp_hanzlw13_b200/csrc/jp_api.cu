@@ -137,6 +137,9 @@ Layout layout(const jp_loop *L) {
   add(R_TLS_S_T, 0);
   add(R_TLS_C_T, tI ? 8 * (size_t)L->len_T : 0);
   add(R_SCHED, sched_layout(L).total);
+  const bool rx = aI && j.op != JP_OP_PRIV_TMP;   // A has exposed reads through an index
+  add(R_MAXRX_A, rx ? 4 * (size_t)L->len_A : 0);
+  add(R_GUIDE, rx ? 8 * (size_t)((L->n + 31) / 32) : 0);
   lo.total = al256(off);
   return lo;
 }
@@ -147,6 +150,7 @@ size_t layout_end(const Layout &lo, int uses) {
   if (uses & JP_WS_PRIV) last = std::max(last, (int)R_KEYS_T);
   if (uses & JP_WS_TLS) last = std::max(last, (int)R_TLS_C_T);
   if (uses & JP_WS_SCHED) last = R_SCHED;
+  if (uses & JP_WS_GUIDE) last = R_GUIDE;
   return al256(lo.off[last] + lo.bytes[last]);
 }
 
@@ -372,6 +376,15 @@ jp_status jp_run_privatized(const jp_loop *L, const jp_profile *p, void *ws, siz
   return jp_priv_finalize(L, ws, ws_bytes, st);
 }
 
+jp_status jp_tls_guide(const jp_loop *L, void *ws, size_t ws_bytes, jp_stream_t st) {
+  JP_TRY(check_loop(L));
+  JP_TRY(need_device());
+  Layout lo;
+  JP_TRY(check_ws(L, ws, ws_bytes, JP_WS_PROFILE | JP_WS_GUIDE, lo));
+  JP_CUDA(launch_tls_guide(make_job(L), ws, lo, (cudaStream_t)st), "tls guide");
+  return JP_OK;
+}
+
 // choose the TLS path and check its limits
 static jp_status tls_plan(const Job &j, const jp_tls_cfg *cfg, const jp_profile *prof, TlsPlan &tp) {
   tp.window = cfg ? cfg->window : 0;
@@ -382,22 +395,54 @@ static jp_status tls_plan(const Job &j, const jp_tls_cfg *cfg, const jp_profile 
   const bool hA = a_indirect(j.op, j.d.r, j.d.r2, j.d.w), hT = t_indirect(j.op, j.d.s);
   tp.waw = (hA || hT) && !(prof && prof->waw_iters == 0);
   const int64_t wcap = tp.window > 0 ? tp.window : tp.w_max;
-  const int64_t cta_max = (j.op == JP_OP_PRIV_TMP && hA && hT) ? kTlsCtaWmax / 2 : kTlsCtaWmax;
   int path = cfg ? cfg->path : 0;
-  if (path == 0) path = wcap <= cta_max ? 1 : 2;
+  int cl = cfg ? cfg->cluster : 0;
+  if (cl < 0 || cl > 16 || (cl & (cl - 1)))
+    return fail(JP_ERR_ARG, "cluster must be 0 (auto) or a power of two <= 16 (got %d)", cl);
+  tp.guided = cfg && cfg->guided;
+  if (tp.guided && (!prof || prof->waw_iters != 0))
+    return fail(JP_ERR_ARG, "a guided TLS run needs a profile with waw_iters == 0");
+  if (tp.guided && !(hA && j.op != JP_OP_PRIV_TMP)) tp.guided = false;   // nothing to guide
+  const int64_t cta_max = tls_cta_wcap(j.op, tp.waw, tp.guided);
+  if (path == 0) {
+    // auto (measured): windows that start small stay on one
+    // SM (a CTA barrier is ~50 cycles, a cluster barrier ~1000); windows that
+    // start at >= 1024 iterations spread their gathers over a 16-CTA cluster
+    // (one SM sustains only ~0.25 random L2/HBM loads per cycle).
+    const int64_t w0 = tp.window > 0 ? tp.window : tls_next_window(j.d.n, tp.prof_raw, -1, tp.w_max);
+    path = w0 < 1024 && wcap <= cta_max ? 1 : wcap <= tls_cluster_wcap(16) ? 3 : 2;
+  }
   if (path == 1 && wcap > cta_max)
     return fail(JP_ERR_UNSUPPORTED, "the single-CTA TLS path holds windows up to %lld iterations", (long long)cta_max);
-  if (path != 1 && path != 2) return fail(JP_ERR_ARG, "bad TLS path %d", path);
+  if (path == 2) tp.guided = false;
+  if (path == 3) {
+    if (cl == 0) cl = tls_max_cluster();   // auto: the largest cluster the device schedules (16 on B200)
+    if (tls_cluster_wcap(cl) < wcap)
+      return fail(JP_ERR_UNSUPPORTED, "a %d-CTA TLS cluster holds windows up to %lld iterations", cl,
+                  (long long)tls_cluster_wcap(cl));
+  }
+  if (path < 1 || path > 3) return fail(JP_ERR_ARG, "bad TLS path %d", path);
+  tp.cluster = cl;
   tp.path = path;
   return JP_OK;
 }
 
+// auto_guide: run jp_tls_guide first when the plan is the cluster path and the
+// profile and workspace allow it (jp_schedule; measured gain at low density)
 static jp_status run_tls_job(const jp_loop *L, const Job &j, const jp_tls_cfg *cfg, const jp_profile *prof, void *ws,
-                             size_t ws_bytes, jp_tls_stats *stats, cudaStream_t st) {
+                             size_t ws_bytes, jp_tls_stats *stats, cudaStream_t st, bool auto_guide = false) {
   TlsPlan tp;
   JP_TRY(tls_plan(j, cfg, prof, tp));
+  if (auto_guide && !tp.guided && tp.path == 3 && prof && prof->waw_iters == 0 && a_indirect(j.op, j.d.r, j.d.r2, j.d.w) &&
+      j.op != JP_OP_PRIV_TMP) {
+    Layout lg = layout(L);
+    if (ws && ws_bytes >= layout_end(lg, JP_WS_PROFILE | JP_WS_GUIDE | JP_WS_TLS) && lg.bytes[R_GUIDE]) {
+      JP_CUDA(launch_tls_guide(j, ws, lg, st), "tls guide");
+      tp.guided = true;
+    }
+  }
   Layout lo;
-  JP_TRY(check_ws(L, ws, ws_bytes, tp.path == 2 ? JP_WS_TLS : 0, lo));
+  JP_TRY(check_ws(L, ws, ws_bytes, (tp.path >= 2 ? JP_WS_TLS : 0) | (tp.guided ? JP_WS_GUIDE : 0), lo));
   if (has_idx(j) && !prof) JP_TRY(validate_sync(j, ws, lo, st, nullptr));
   int64_t *hdr = at<int64_t>(ws, lo, R_HEADER);
   JP_CUDA(launch_tls(j, ws, lo, tp, &hdr[H_TLS_COMMITTED], st), "tls");
@@ -419,6 +464,10 @@ jp_status jp_run_tls(const jp_loop *L, const jp_tls_cfg *cfg, const jp_profile *
   JP_TRY(need_device());
   return run_tls_job(L, make_job(L), cfg, prof, ws, ws_bytes, stats, (cudaStream_t)st);
 }
+
+#ifdef JP_TLS_TRACE
+int32_t jp_tls_trace(long long *host, int32_t n) { return (int32_t)jp::tls_trace_copy(host, n); }
+#endif
 
 jp_status jp_merge_apply(void *arr, int64_t len, const int64_t *keys, jp_stream_t st) {
   if (len < 0 || (len > 0 && (!arr || !keys))) return fail(JP_ERR_ARG, "bad merge arguments");
@@ -551,8 +600,9 @@ static jp_status run_mode(const jp_loop *L, const Job &j, int mode, const jp_pro
     JP_CUDA(launch_priv_stream(j, ws, lo, true, st), "priv stream");
     JP_CUDA(launch_priv_finalize(j, ws, lo, st), "priv finalize");
   } else {
-    jp_tls_cfg tc{c.tls_window, c.tls_w_max, c.tls_path, 0};
-    JP_TRY(run_tls_job(L, j, &tc, prof, ws, ws_bytes, &res->tls, st));
+    // profile-guided mode B on the cluster path
+    jp_tls_cfg tc{c.tls_window, c.tls_w_max, c.tls_path, 0, 0, 0};
+    JP_TRY(run_tls_job(L, j, &tc, prof, ws, ws_bytes, &res->tls, st, true));
   }
   res->task_mode_iters[mode] += j.d.n;
   return JP_OK;
@@ -671,7 +721,7 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
         Job sj = sub_job(j, tasks[t].s, tasks[t].e);
         if (tls) {
           TlsPlan tp;
-          jp_tls_cfg tc{c.tls_window, c.tls_w_max, 1, 0};
+          jp_tls_cfg tc{c.tls_window, c.tls_w_max, 1, 0, 0, 0};
           jp_profile tprof{};
           tprof.n = sj.d.n;
           tprof.raw_iters = hc.empty() ? -1 : 0;

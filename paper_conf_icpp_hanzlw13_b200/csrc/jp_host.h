@@ -10,7 +10,7 @@ namespace jp {
 enum Region : int {
   R_HEADER = 0, R_MINW_A = 1, R_MINR_A = 2, R_MINW_T = 3, R_MINR_T = 4, R_KEYS_A = 5,
   R_KEYS_T = 6, R_TLS_S_A = 7, R_TLS_C_A = 8, R_TLS_S_T = 9, R_TLS_C_T = 10, R_SCHED = 11,
-  R_COUNT = 12
+  R_MAXRX_A = 12, R_GUIDE = 13, R_COUNT = 14
 };
 
 struct Layout {
@@ -44,6 +44,9 @@ Job make_job(const jp_loop *L);
 
 // ---- launchers (each returns the first CUDA error, if any) ----
 cudaError_t launch_validate(const Job &j, int64_t *hdr, cudaStream_t st);
+// TLS guide bitmaps (region R_GUIDE: raw words then source words) from the
+// stamp tables of a profile on the same workspace; no sync.
+cudaError_t launch_tls_guide(const Job &j, void *ws, const Layout &lo, cudaStream_t st);
 cudaError_t launch_prof_stamp(const Job &j, void *ws, const Layout &lo, cudaStream_t st);
 cudaError_t launch_prof_classify(const Job &j, void *ws, const Layout &lo, uint32_t *raw_bits,
                                  int64_t chunk, int64_t *chunk_counts, cudaStream_t st);
@@ -63,12 +66,20 @@ cudaError_t launch_task_conflicts(const Job &j, const int32_t *chunk_task, int64
 struct TlsPlan {
   int64_t window, w_max, prof_raw;  // prof_raw < 0: no profile
   bool waw;                         // in-window WAW resolution needed
-  int path;                         // 1 cta, 2 grid
+  int path;                         // 1 cta, 2 grid, 3 cluster
+  int cluster;                      // CTAs of the cluster path (power of two)
+  bool guided;                      // stamp only RAW sources, check only RAW readers
 };
 // stats: int64[4] device (committed, executed, windows, violations); bar: u32[2]
 // zeroed barrier words + int64[3] fv slots (grid path).
 cudaError_t launch_tls(const Job &j, void *ws, const Layout &lo, const TlsPlan &p, int64_t *stats,
                        cudaStream_t st);
 int64_t tls_next_window(int64_t n, int64_t prof_raw, int64_t prev_commit, int64_t w_max);
+int64_t tls_cluster_wcap(int cluster);
+int64_t tls_cta_wcap(int op, bool waw, bool guided);   // largest single-CTA window
+int tls_max_cluster();                                 // 16 when the device schedules it, else 8
+#ifdef JP_TLS_TRACE
+cudaError_t tls_trace_copy(long long *host, int n);
+#endif
 
 }  // namespace jp

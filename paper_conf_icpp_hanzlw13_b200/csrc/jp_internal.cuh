@@ -17,10 +17,10 @@ namespace jp {
 
 constexpr int kSmemSlots = 4096;          // arrays this small are pre-aggregated per CTA
 #ifndef JP_TLS_THREADS
-#define JP_TLS_THREADS 1024
+#define JP_TLS_THREADS 512
 #endif
 #ifndef JP_TLS_IPT
-#define JP_TLS_IPT 4
+#define JP_TLS_IPT 8
 #endif
 #ifndef JP_TLS_HASHLOG
 #define JP_TLS_HASHLOG 13

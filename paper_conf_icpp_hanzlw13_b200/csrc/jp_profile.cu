@@ -157,6 +157,66 @@ __global__ void __launch_bounds__(256) k_prof_classify(DLoop L, Tabs t, uint32_t
   if (threadIdx.x == 0 && s_first != ~0ull) atomicMin((unsigned long long *)&hdr[H_FIRST_RAW], s_first);
 }
 
+// ---------------------------------------------------------------------------
+// TLS guide (profile-guided mode B).  Two bitmaps over
+// local iterations, one bit per iteration, 32 iterations per word:
+//   raw_i  some exposed read a of i has an earlier writer (minW table, pass 1);
+//   src_j  the A-write of j is exposed-read by a later iteration (maxRx table).
+// An in-window RAW violation needs a raw reader and a source writer (reading
+// A7), so TLS windows stamp only source writes and check only raw reads: the
+// same first violator, hence the same windows and statistics.
+// Pass G1 fills maxRx[a] = latest gid with an exposed read of a (int32, empty
+// -1): __match_any_sync groups the lanes of a warp that read the same address
+// and only the group's highest lane (its latest iteration) issues the atomic.
+template <int OP>
+__global__ void __launch_bounds__(256) k_guide_maxr(DLoop L, int32_t *maxRx) {
+  const int64_t stride = (int64_t)gridDim.x * blockDim.x;
+  const int64_t n_up = (L.n + 31) & ~(int64_t)31;   // whole warps for the match
+  const int lane = threadIdx.x & 31;
+  for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n_up; i += stride) {
+    const bool act = i < L.n;
+    const int32_t g = (int32_t)(L.base + i);
+    int32_t a0 = -1, a1 = -1;
+    if (act) {
+      if constexpr (OP == JP_OP_SAXPY) a0 = (int32_t)ixl(L, L.w, i);
+      else if constexpr (OP == JP_OP_ADD_C) a0 = (int32_t)ixl(L, L.r, i);
+      else if constexpr (OP == JP_OP_STENCIL2) { a0 = (int32_t)ixl(L, L.r, i); a1 = (int32_t)ixl(L, L.r2, i); }
+    }
+    if constexpr (OP != JP_OP_PRIV_TMP) {
+      const unsigned grp = __match_any_sync(0xffffffffu, a0);
+      if (act && (31 - __clz(grp)) == lane) atomicMax(&maxRx[a0], g);
+      if constexpr (OP == JP_OP_STENCIL2) {
+        const unsigned grp2 = __match_any_sync(0xffffffffu, a1);
+        if (act && (31 - __clz(grp2)) == lane) atomicMax(&maxRx[a1], g);
+      }
+    }
+  }
+}
+
+// Pass G2: the two bitmaps (ballot per warp tile).
+template <int OP>
+__global__ void __launch_bounds__(256) k_guide_bits(DLoop L, const int32_t *minW, const int32_t *maxRx,
+                                                    uint32_t *raw_bits, uint32_t *src_bits) {
+  const int lane = threadIdx.x & 31;
+  const int64_t warps = (int64_t)gridDim.x * (blockDim.x >> 5);
+  const int64_t tiles = (L.n + 31) >> 5;
+  for (int64_t tile = (int64_t)blockIdx.x * (blockDim.x >> 5) + (threadIdx.x >> 5); tile < tiles; tile += warps) {
+    const int64_t i = (tile << 5) + lane;
+    bool raw = false, src = false;
+    if (i < L.n && OP != JP_OP_PRIV_TMP) {
+      const int64_t gid = L.base + i;
+      const int32_t e = enc_gid(gid);
+      const int64_t a = ixl(L, L.w, i);
+      if constexpr (OP == JP_OP_SAXPY) raw = minW[a] > e;
+      else raw = minW[ixl(L, L.r, i)] > e;
+      if constexpr (OP == JP_OP_STENCIL2) raw = raw || minW[ixl(L, L.r2, i)] > e;
+      src = maxRx[a] > (int32_t)gid;
+    }
+    const unsigned bR = __ballot_sync(0xffffffffu, raw), bS = __ballot_sync(0xffffffffu, src);
+    if (lane == 0) { raw_bits[tile] = bR; src_bits[tile] = bS; }
+  }
+}
+
 template <int OP>
 __global__ void __launch_bounds__(256) k_validate(DLoop L, int64_t *hdr) {
   int64_t bad = 0;
@@ -242,6 +302,25 @@ static void run_validate(const DLoop &d, int64_t *hdr, cudaStream_t st) {
   (void)DT;
   k_validate<OP><<<grid_for(d.n, 256, 8), 256, 0, st>>>(d, hdr);
   note_launch();
+}
+
+template <int OP, int DT>
+static void run_guide(const DLoop &d, int32_t *minW, int32_t *maxRx, uint32_t *bits, cudaStream_t st) {
+  (void)DT;
+  const int64_t nw = (d.n + 31) / 32;
+  k_guide_maxr<OP><<<grid_for(d.n, 256, 8), 256, 0, st>>>(d, maxRx);
+  k_guide_bits<OP><<<grid_for(nw * 32, 256, 8), 256, 0, st>>>(d, minW, maxRx, bits, bits + nw);
+  note_launch(2);
+}
+
+cudaError_t launch_tls_guide(const Job &j, void *ws, const Layout &lo, cudaStream_t st) {
+  int32_t *maxRx = at<int32_t>(ws, lo, R_MAXRX_A);
+  uint32_t *bits = at<uint32_t>(ws, lo, R_GUIDE);
+  int32_t *minW = at<int32_t>(ws, lo, R_MINW_A);
+  if (!bits || !maxRx || !minW || j.d.n == 0) return launch_check();
+  cudaMemsetAsync(maxRx, 0xFF, lo.bytes[R_MAXRX_A], st);
+  JP_DISPATCH(j.op, j.dt, run_guide, j.d, minW, maxRx, bits, st);
+  return launch_check();
 }
 
 cudaError_t launch_validate(const Job &j, int64_t *hdr, cudaStream_t st) {

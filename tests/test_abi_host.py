@@ -47,9 +47,9 @@ def cpu_loop(op=0, n=1000, la=1000, r=True, w=True, s=False, lt=16):
 
 def test_workspace_layout_fixed_offsets():
     L = cpu_loop()
-    sizes = {u: jp.jp_workspace_bytes(L, u) for u in (0, 1, 2, 4, 8, 15)}
+    sizes = {u: jp.jp_workspace_bytes(L, u) for u in (0, 1, 2, 4, 8, 15, 16, 31)}
     assert sizes[0] == 4096
-    assert sizes[1] < sizes[2] < sizes[4] < sizes[8] == sizes[15]
+    assert sizes[1] < sizes[2] < sizes[4] < sizes[8] == sizes[15] < sizes[16] == sizes[31]
     # regions are disjoint, 256-aligned and inside the total
     spans = []
     for name in _abi.REGIONS:
@@ -57,7 +57,7 @@ def test_workspace_layout_fixed_offsets():
         assert off % 256 == 0
         if nb:
             spans.append((off, off + nb))
-            assert off + nb <= sizes[15]
+            assert off + nb <= sizes[31]
     spans.sort()
     for a, b in zip(spans, spans[1:]):
         assert a[1] <= b[0]
@@ -67,6 +67,9 @@ def test_workspace_layout_fixed_offsets():
     Lt = cpu_loop(op=2, r=False, w=False, s=True, lt=1024)
     assert jp.jp_ws_region(Lt, "minW_T")[1] == 4 * 1024 and jp.jp_ws_region(Lt, "keys_T")[1] == 8 * 1024
     assert jp.jp_ws_region(Lt, "keys_A")[1] == 0
+    # guide regions: maxRx over A and two bitmaps of ceil(n/32) words (opcodes with exposed A reads)
+    assert jp.jp_ws_region(L, "maxRx_A")[1] == 4 * 1000 and jp.jp_ws_region(L, "guide")[1] == 8 * 32
+    assert jp.jp_ws_region(Lt, "guide")[1] == 0
 
 
 @pytest.mark.parametrize("seed", range(200))

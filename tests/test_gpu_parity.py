@@ -322,15 +322,17 @@ def test_config4_full_size():
 # ---------------------------------------------------------------------------
 # TLS
 # ---------------------------------------------------------------------------
-def tls_case(wl, window, path, w_max=65536, with_prof=False):
+def tls_case(wl, window, path, w_max=65536, with_prof=False, cluster=0, guided=False):
     ref = to_oracle(wl)
-    prof_raw = O.profile(ref)["raw_iters"] if with_prof else -1
+    prof_raw = O.profile(ref)["raw_iters"] if (with_prof or guided) else -1
     st, A, T, stats = O.sim_tls(ref, window, w_max, prof_raw)
     g = gpu(wl)
     L = jp.Loop.from_workload(g)
     ws = jp.workspace(L)
-    p = jp.jp_profile_density(L, ws) if with_prof else None
-    got = jp.jp_run_tls(L, window=window, w_max=w_max, path=path, prof=p, ws=ws)
+    p = jp.jp_profile_density(L, ws) if (with_prof or guided) else None
+    if guided:
+        jp.jp_tls_guide(L, ws)
+    got = jp.jp_run_tls(L, window=window, w_max=w_max, path=path, prof=p, ws=ws, cluster=cluster, guided=guided)
     torch.cuda.synchronize()
     check_arrays(g, A, T)
     assert got == stats, (got, stats)
@@ -338,14 +340,14 @@ def tls_case(wl, window, path, w_max=65536, with_prof=False):
 
 
 @pytest.mark.parametrize("window,path", [(32, 1), (100, 1), (1024, 1), (4096, 1), (32, 2), (1000, 2), (8192, 2),
-                                         (65536, 2)])
+                                         (65536, 2), (32, 3), (100, 3), (1000, 3), (4096, 3), (65536, 3)])
 @pytest.mark.parametrize("d", [0.0, 0.05])
 def test_tls_config1(window, path, d):
     tls_case(synth.config1(d), window, path)
 
 
 @pytest.mark.parametrize("d", [0.001, 0.01, 0.10])
-@pytest.mark.parametrize("path", [1, 2])
+@pytest.mark.parametrize("path", [1, 2, 3])
 def test_tls_config3_reduced(d, path):
     tls_case(synth.config3(d, n=(1 << 17) + 11), 4096, path)
 
@@ -354,13 +356,13 @@ def test_tls_config3_reduced(d, path):
 def test_tls_random(op, dt, seed):
     n = [200, 3000, 9001][seed]
     wl = random_loop(500 + op * 10 + dt * 3 + seed, op, dt, n, len_a=max(32, n // [1, 4, 2][seed]))
-    for window, path in ((64, 1), (1000, 1), (1000, 2)):
+    for window, path in ((64, 1), (1000, 1), (1000, 2), (64, 3), (1000, 3)):
         if op == O.OP_PRIV_TMP and window > 2048 and path == 1:
             continue
         tls_case(wl, window, path)
 
 
-@pytest.mark.parametrize("path", [1, 2])
+@pytest.mark.parametrize("path", [1, 2, 3])
 def test_tls_adaptive(path):
     wl = synth.config3(0.01, n=1 << 16)
     w_max = 4096 if path == 1 else 65536
@@ -384,6 +386,125 @@ def test_tls_gauss_seidel_and_prefix_chain():
 def test_config3_full_size_stats():
     """BASELINE size N=2^24 at d=1%, W=4096 (bench configuration): full arrays and stats."""
     tls_case(synth.config3(0.01), 4096, 1)
+    tls_case(synth.config3(0.01), 4096, 3)
+
+
+@pytest.mark.parametrize("cluster", [1, 2, 4, 8, 16])
+def test_tls_cluster_sizes(cluster):
+    """The cluster path at every cluster size (incl. a non power of two), fixed
+    and adaptive windows, with and without the WAW commit (profile or not)."""
+    wl = synth.config3(0.05, n=(1 << 15) + 77)
+    for window in (96, 1000, 4096):
+        if window <= 32 * (144 * cluster - 1):
+            tls_case(wl, window, 3, cluster=cluster)
+            tls_case(wl, window, 3, cluster=cluster, with_prof=True)
+    tls_case(wl, 0, 3, w_max=4096, cluster=cluster, with_prof=True)
+
+
+@pytest.mark.parametrize("op,dt", [(op, dt) for op in OPS for dt in DTS])
+def test_tls_cluster_waw_unaligned(op, dt):
+    """In-window WAW (many writers per address, len_A = 64) and index streams
+    that are not 16-byte aligned (views starting 3 entries in): the 4-byte ring
+    fill and the __match_any_sync commit groups of the cluster path."""
+    n = 5000
+    wl = random_loop(900 + op * 10 + dt, op, dt, n + 3, len_a=64, null_prob=0.0)
+    sl = lambda t: None if t is None else t[3:]  # noqa: E731
+    sub = synth.Workload("sub", wl.op, wl.dtype, n, wl.A.clone(), r=sl(wl.r), r2=sl(wl.r2), w=sl(wl.w),
+                         s=sl(wl.s), X=wl.X, T=None if wl.T is None else wl.T.clone(), c0=wl.c0, c1=wl.c1)
+    for window in (64, 1000):
+        _, A, T, stats = O.sim_tls(to_oracle(sub), window, 65536, -1)
+        g = gpu(wl)
+        L = jp.Loop(wl.op, wl.dtype, n, g.A, r=sl(g.r), w=sl(g.w), r2=sl(g.r2), s=sl(g.s), X=g.X, T=g.T,
+                    c0=wl.c0, c1=wl.c1)
+        got = jp.jp_run_tls(L, window=window, path=3, ws=jp.workspace(L))
+        torch.cuda.synchronize()
+        check_arrays(g, A, T)
+        assert got == stats, (window, got, stats)
+
+
+def test_tls_cluster_size_must_be_pow2():
+    wl = gpu(synth.config1(0.05))
+    L = jp.Loop.from_workload(wl)
+    with pytest.raises(jp.JPError):
+        jp.jp_run_tls(L, window=64, path=3, cluster=3, ws=jp.workspace(L))
+
+
+# ---------------------------------------------------------------------------
+# profile-guided TLS (SURVEY Sec.8(f) NEXT-1)
+# ---------------------------------------------------------------------------
+def guide_case(wl):
+    """The guide bitmaps equal the oracle's raw flags and RAW-source flags."""
+    ref = to_oracle(wl)
+    g = gpu(wl)
+    L = jp.Loop.from_workload(g)
+    ws = jp.workspace(L)
+    jp.jp_profile_density(L, ws)
+    jp.jp_tls_guide(L, ws)
+    torch.cuda.synchronize()
+    off, nb = jp.jp_ws_region(L, "guide")
+    nw = (wl.n + 31) // 32
+    words = ws[off:off + 8 * nw].view(torch.int32)
+    raw = bits_to_flags(words[:nw], wl.n)
+    src = bits_to_flags(words[nw:], wl.n)
+    assert np.array_equal(raw, O.profile(ref)["flags"] & 1)
+    assert np.array_equal(src, O.raw_sources(ref))
+
+
+@pytest.mark.parametrize("op,dt,seed", [(op, dt, s) for op in (O.OP_ADD_C, O.OP_SAXPY, O.OP_STENCIL2)
+                                        for dt in DTS for s in range(2)])
+def test_guide_bits_random(op, dt, seed):
+    n = [777, 5000][seed]
+    guide_case(random_loop(700 + op * 10 + dt * 3 + seed, op, dt, n, len_a=max(64, n // 3), null_prob=0.0))
+
+
+@pytest.mark.parametrize("d", [0.0, 0.001, 0.05, 0.10])
+def test_guide_bits_config3(d):
+    guide_case(synth.config3(d, n=(1 << 16) + 9))
+
+
+@pytest.mark.parametrize("path", [1, 3])
+@pytest.mark.parametrize("d", [0.001, 0.01, 0.05, 0.10])
+def test_tls_guided_config3_reduced(d, path):
+    wl = synth.config3(d, n=(1 << 17) + 11)
+    for window in (96, 1000, 4096):
+        tls_case(wl, window, path, guided=True)
+    tls_case(wl, 0, path, w_max=4096, guided=True)
+
+
+@pytest.mark.parametrize("op,dt", [(op, dt) for op in (O.OP_ADD_C, O.OP_SAXPY, O.OP_STENCIL2) for dt in DTS])
+def test_tls_guided_random_waw_free(op, dt):
+    """Write-once loops (w a partial permutation: no WAW) of every opcode with
+    exposed reads, guided on both paths; the result equals the unguided run."""
+    n = 6000
+    wl = random_loop(300 + op * 10 + dt, op, dt, n, len_a=3 * n, null_prob=0.0, dup_writes=False)
+    for path in (1, 3):
+        for window in (64, 1500):
+            tls_case(wl, window, path, guided=True)
+
+
+def test_tls_guided_needs_waw_free_profile():
+    wl = gpu(random_loop(5, O.OP_ADD_C, O.I32, 3000, len_a=64, null_prob=0.0))
+    L = jp.Loop.from_workload(wl)
+    ws = jp.workspace(L)
+    p = jp.jp_profile_density(L, ws)
+    assert p["waw_iters"] > 0
+    with pytest.raises(jp.JPError):
+        jp.jp_run_tls(L, window=64, prof=p, ws=ws, guided=True)
+
+
+@pytest.mark.parametrize("d", [0.01, 0.10])
+def test_config3_full_size_guided(d):
+    """BASELINE size N=2^24 through jp_schedule (profile -> guide -> TLS), full arrays and stats."""
+    wl = synth.config3(d)
+    ref = to_oracle(wl)
+    _, A, _, stats = O.sim_tls(ref, 0, 4096, O.profile(ref)["raw_iters"])
+    g = gpu(wl)
+    L = jp.Loop.from_workload(g)
+    res = jp.jp_schedule(L, jp.workspace(L))
+    torch.cuda.synchronize()
+    assert res["mode"] == jp.JP_MODE_TLS
+    check_arrays(g, A, None)
+    assert res["tls"] == stats, (res["tls"], stats)
 
 
 # ---------------------------------------------------------------------------
