@@ -23,7 +23,7 @@ from ._abi import (  # noqa: F401
 __all__ = [
     "Loop", "workspace", "jp_workspace_bytes", "jp_ws_region", "jp_validate", "jp_profile_stamp",
     "jp_profile_classify", "jp_profile_density", "jp_select_mode", "jp_run_doall", "jp_run_privatized",
-    "jp_priv_stream", "jp_priv_finalize", "jp_tls_guide", "jp_run_tls", "jp_schedule", "jp_stage_bytes", "jp_schedule_host",
+    "jp_priv_stream", "jp_priv_finalize", "jp_tls_guide", "tls_first_window", "jp_run_tls", "jp_schedule", "jp_stage_bytes", "jp_schedule_host",
     "jp_plan_sharing", "jp_plan_stealing", "jp_merge_apply", "jp_last_error", "jp_version", "jp_launch_count",
 ]
 
@@ -191,6 +191,19 @@ def jp_priv_stream(loop: Loop, prof=None, ws=None, clear_keys=True, stream=None)
 def jp_priv_finalize(loop: Loop, ws, stream=None):
     p, nb = _ws(ws)
     check(lib().jp_priv_finalize(loop.ref, p, nb, _stream(stream)))
+
+
+def tls_first_window(n: int, raw_iters: int, w_max: int = 4096) -> int:
+    """Reading A8's first adaptive window (jp.h): clamp(pow2ceil(ceil(4n/raw)), 32, w_max),
+    w_max when raw == 0, 4096 without a profile (raw < 0).  Host arithmetic only."""
+    if raw_iters < 0:
+        w0 = 4096
+    elif raw_iters == 0:
+        w0 = w_max
+    else:
+        q = (4 * n + raw_iters - 1) // raw_iters
+        w0 = 1 << max(0, (q - 1).bit_length())
+    return max(32, min(w0, w_max))
 
 
 def jp_tls_guide(loop: Loop, ws: torch.Tensor, stream=None) -> None:

@@ -10,8 +10,11 @@
 //   with a check-before-atomic filter; ascending gid order inside a CTA makes
 //   every touch after the first a no-op.
 // Pass 2 (classify): per iteration raw/war/waw against the tables (reading
-//   A1), then __ballot_sync + __popc per warp, one shared atomic per warp, one
-//   global atomic per CTA; optional raw bitmap (D4) and per-chunk counts.
+//   A1).  Counts only (jp_schedule's call): per-thread counters, one warp
+//   reduction and one global atomic per CTA.  With a raw bitmap (D4) or
+//   per-chunk counts: __ballot_sync + __popc per warp tile of 32 iterations.
+// Both passes take 4 consecutive iterations per thread (16-byte index loads)
+// with two steps in flight and 32-bit index arithmetic.
 // The intra-warp / inter-warp split of the paper is an
 // implementation detail here (reading A2): results do not depend on geometry.
 #include "jp_host.h"
@@ -23,57 +26,109 @@ struct Tabs {
   int sA, sT;   // pre-aggregate in shared memory
 };
 
-__device__ __forceinline__ void stamp(int32_t *g, int32_t *s, int64_t a, int64_t len, int32_t e, int64_t &bad) {
-  if ((uint64_t)a >= (uint64_t)len) { bad++; return; }
+__device__ __forceinline__ void check(int64_t a, int64_t len, int64_t &bad) {
+  if ((uint64_t)a >= (uint64_t)len) bad++;
+}
+
+// Loads of kUnroll iterations (one per CTA-wide slice) are issued before any
+// of them is used: the passes stream their index arrays from HBM, and one
+// dependent load chain per warp at a time would leave them latency-bound.
+constexpr int kUnroll = 4;
+
+// ---------------------------------------------------------------------------
+// Quad variants: each thread takes 4 consecutive iterations per step (one
+// 16-byte load per index stream when every stream is 16-byte aligned), two
+// steps in flight, 32-bit index arithmetic.  Same tables, same counts.
+// ---------------------------------------------------------------------------
+__device__ __forceinline__ int4 idx4(const DLoop &L, const int32_t *p, int64_t i, bool vec) {
+  if (!p) {
+    const int b = (int)(L.ioff + i);
+    return make_int4(b, b + 1, b + 2, b + 3);
+  }
+  if (vec && i + 4 <= L.n) return __ldcs(reinterpret_cast<const int4 *>(p + i));
+  int4 r;
+  r.x = p[i];
+  r.y = i + 1 < L.n ? p[i + 1] : 0;
+  r.z = i + 2 < L.n ? p[i + 2] : 0;
+  r.w = i + 3 < L.n ? p[i + 3] : 0;
+  return r;
+}
+__device__ __forceinline__ int q4(const int4 &v, int k) { return k == 0 ? v.x : k == 1 ? v.y : k == 2 ? v.z : v.w; }
+__device__ __forceinline__ void stamp32(int32_t *g, int32_t *s, int32_t a, int32_t len, int32_t e, int &bad) {
+  if ((uint32_t)a >= (uint32_t)len) { bad++; return; }
   if (s) {
     if (s[a] < e) atomicMax(&s[a], e);
   } else if (g) {
     atomicMax(&g[a], e);
   }
 }
-__device__ __forceinline__ void check(int64_t a, int64_t len, int64_t &bad) {
-  if ((uint64_t)a >= (uint64_t)len) bad++;
+__device__ __forceinline__ bool earlier32(const int32_t *tab, int32_t a, int32_t len, int32_t e) {
+  return tab && (uint32_t)a < (uint32_t)len && tab[a] > e;
 }
+constexpr int kQuadSteps = 2;
 
 template <int OP>
-__global__ void __launch_bounds__(256) k_prof_stamp(DLoop L, Tabs t, int64_t *hdr) {
+__global__ void __launch_bounds__(256) k_prof_stamp4(DLoop L, Tabs t, int vec, int64_t *hdr) {
   extern __shared__ int32_t sm[];
-  int32_t *sAw = nullptr, *sAr = nullptr, *sTw = nullptr, *sTr = nullptr;
+  int32_t *sAw = nullptr, *sAr = nullptr, *sTw = nullptr;
   int32_t *p = sm;
   if (t.sA) { sAw = p; p += L.lenA; if (t.rA) { sAr = p; p += L.lenA; } }
-  if (t.sT) { sTw = p; p += L.lenT; sTr = p; p += L.lenT; }
+  if (t.sT) { sTw = p; p += L.lenT; }   // minR(T) == minW(T) for PRIV_TMP (see k_prof_stamp)
   for (int64_t k = threadIdx.x; k < p - sm; k += blockDim.x) sm[k] = -1;
   JP_CTA_SYNC();
-
-  int64_t bad = 0;
-  const int64_t stride = (int64_t)gridDim.x * blockDim.x;
-  for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < L.n; i += stride) {
-    const int32_t e = enc_gid(L.base + i);
-    if constexpr (OP == JP_OP_ADD_C) {
-      stamp(t.wA, sAw, ixl(L, L.w, i), L.lenA, e, bad);
-      stamp(t.rA, sAr, ixl(L, L.r, i), L.lenA, e, bad);
-    } else if constexpr (OP == JP_OP_SAXPY) {
-      check(ixl(L, L.r, i), L.lenX, bad);
-      int64_t a = ixl(L, L.w, i);
-      stamp(t.wA, sAw, a, L.lenA, e, bad);
-      if ((uint64_t)a < (uint64_t)L.lenA) stamp(t.rA, sAr, a, L.lenA, e, bad);
-    } else if constexpr (OP == JP_OP_PRIV_TMP) {
-      check(ixl(L, L.r, i), L.lenX, bad);
-      int64_t a = ixl(L, L.s, i);
-      stamp(t.wT, sTw, a, L.lenT, e, bad);
-      if ((uint64_t)a < (uint64_t)L.lenT) stamp(t.rT, sTr, a, L.lenT, e, bad);
-      stamp(t.wA, sAw, ixl(L, L.w, i), L.lenA, e, bad);
-    } else {
-      stamp(t.wA, sAw, ixl(L, L.w, i), L.lenA, e, bad);
-      stamp(t.rA, sAr, ixl(L, L.r, i), L.lenA, e, bad);
-      stamp(t.rA, sAr, ixl(L, L.r2, i), L.lenA, e, bad);
+  const int32_t lenA = (int32_t)L.lenA, lenX = (int32_t)L.lenX, lenT = (int32_t)L.lenT;
+  int bad = 0;
+  const int64_t nq = (L.n + 3) >> 2, B = blockDim.x;
+  for (int64_t q0 = (int64_t)blockIdx.x * B * kQuadSteps + threadIdx.x; q0 < nq; q0 += (int64_t)gridDim.x * B * kQuadSteps) {
+    int4 va[kQuadSteps], vb[kQuadSteps], vc[kQuadSteps];
+#pragma unroll
+    for (int u = 0; u < kQuadSteps; u++) {
+      const int64_t q = q0 + u * B;
+      if (q < nq) {
+        const int64_t i = q << 2;
+        if constexpr (OP == JP_OP_ADD_C || OP == JP_OP_SAXPY) { va[u] = idx4(L, L.w, i, vec); vb[u] = idx4(L, L.r, i, vec); }
+        else if constexpr (OP == JP_OP_PRIV_TMP) { va[u] = idx4(L, L.s, i, vec); vb[u] = idx4(L, L.r, i, vec); vc[u] = idx4(L, L.w, i, vec); }
+        else { va[u] = idx4(L, L.w, i, vec); vb[u] = idx4(L, L.r, i, vec); vc[u] = idx4(L, L.r2, i, vec); }
+      }
+    }
+#pragma unroll
+    for (int u = 0; u < kQuadSteps; u++) {
+      const int64_t q = q0 + u * B;
+      if (q >= nq) break;
+      const int32_t e0 = enc_gid(L.base + (q << 2));
+      const int kn = L.n - (q << 2) < 4 ? (int)(L.n - (q << 2)) : 4;
+#pragma unroll
+      for (int k = 0; k < 4; k++) {
+        if (k >= kn) break;
+        const int32_t e = e0 - k;
+        const int32_t a = q4(va[u], k), b = q4(vb[u], k);
+        if constexpr (OP == JP_OP_ADD_C) {
+          stamp32(t.wA, sAw, a, lenA, e, bad);
+          stamp32(t.rA, sAr, b, lenA, e, bad);
+        } else if constexpr (OP == JP_OP_SAXPY) {
+          if ((uint32_t)b >= (uint32_t)lenX) bad++;
+          stamp32(t.wA, sAw, a, lenA, e, bad);
+          if ((uint32_t)a < (uint32_t)lenA) stamp32(t.rA, sAr, a, lenA, e, bad);
+        } else if constexpr (OP == JP_OP_PRIV_TMP) {
+          if ((uint32_t)b >= (uint32_t)lenX) bad++;
+          if (sTw) {
+            stamp32(t.wT, sTw, a, lenT, e, bad);
+          } else {
+            stamp32(t.wT, nullptr, a, lenT, e, bad);
+            if ((uint32_t)a < (uint32_t)lenT) stamp32(t.rT, nullptr, a, lenT, e, bad);
+          }
+          stamp32(t.wA, sAw, q4(vc[u], k), lenA, e, bad);
+        } else {
+          stamp32(t.wA, sAw, a, lenA, e, bad);
+          stamp32(t.rA, sAr, b, lenA, e, bad);
+          stamp32(t.rA, sAr, q4(vc[u], k), lenA, e, bad);
+        }
+      }
     }
   }
-  // warp-aggregate the bad-index count
-  for (int o = 16; o; o >>= 1) bad += __shfl_xor_sync(0xffffffffu, bad, o);
+  bad = __reduce_add_sync(0xffffffffu, bad);
   if ((threadIdx.x & 31) == 0 && bad) atomicAdd((unsigned long long *)&hdr[H_BAD], (unsigned long long)bad);
   JP_CTA_SYNC();
-  // flush the per-CTA pre-aggregated tables
   if (t.sA) {
     for (int64_t a = threadIdx.x; a < L.lenA; a += blockDim.x) {
       if (sAw[a] != -1) atomicMax(&t.wA[a], sAw[a]);
@@ -81,11 +136,92 @@ __global__ void __launch_bounds__(256) k_prof_stamp(DLoop L, Tabs t, int64_t *hd
     }
   }
   if (t.sT) {
-    for (int64_t a = threadIdx.x; a < L.lenT; a += blockDim.x) {
-      if (sTw[a] != -1) atomicMax(&t.wT[a], sTw[a]);
-      if (sTr[a] != -1) atomicMax(&t.rT[a], sTr[a]);
+    for (int64_t a = threadIdx.x; a < L.lenT; a += blockDim.x)
+      if (sTw[a] != -1) { atomicMax(&t.wT[a], sTw[a]); atomicMax(&t.rT[a], sTw[a]); }
+  }
+}
+
+// counts-only classify (no raw bitmap, no chunk counts): per-thread counters,
+// one reduction per CTA
+template <int OP>
+__global__ void __launch_bounds__(256) k_prof_count4(DLoop L, Tabs t, int vec, int64_t *hdr) {
+  __shared__ unsigned long long s_cnt[3];
+  __shared__ unsigned long long s_first;
+  if (threadIdx.x < 3) s_cnt[threadIdx.x] = 0;
+  if (threadIdx.x == 0) s_first = ~0ull;
+  JP_CTA_SYNC();
+  const int32_t lenA = (int32_t)L.lenA, lenT = (int32_t)L.lenT;
+  const int32_t *rT = OP == JP_OP_PRIV_TMP ? t.wT : t.rT;
+  unsigned c_raw = 0, c_war = 0, c_waw = 0;
+  unsigned long long first = ~0ull;
+  const int64_t nq = (L.n + 3) >> 2, B = blockDim.x;
+  for (int64_t q0 = (int64_t)blockIdx.x * B * kQuadSteps + threadIdx.x; q0 < nq; q0 += (int64_t)gridDim.x * B * kQuadSteps) {
+    int4 va[kQuadSteps], vb[kQuadSteps], vc[kQuadSteps];
+#pragma unroll
+    for (int u = 0; u < kQuadSteps; u++) {
+      const int64_t q = q0 + u * B;
+      if (q < nq) {
+        const int64_t i = q << 2;
+        if constexpr (OP == JP_OP_ADD_C) { va[u] = idx4(L, L.w, i, vec); vb[u] = idx4(L, L.r, i, vec); }
+        else if constexpr (OP == JP_OP_SAXPY) { va[u] = idx4(L, L.w, i, vec); }
+        else if constexpr (OP == JP_OP_PRIV_TMP) { va[u] = idx4(L, L.s, i, vec); vb[u] = idx4(L, L.w, i, vec); }
+        else { va[u] = idx4(L, L.w, i, vec); vb[u] = idx4(L, L.r, i, vec); vc[u] = idx4(L, L.r2, i, vec); }
+      }
+    }
+#pragma unroll
+    for (int u = 0; u < kQuadSteps; u++) {
+      const int64_t q = q0 + u * B;
+      if (q >= nq) break;
+      const int32_t e0 = enc_gid(L.base + (q << 2));
+      const int kn = L.n - (q << 2) < 4 ? (int)(L.n - (q << 2)) : 4;
+#pragma unroll
+      for (int k = 0; k < 4; k++) {
+        if (k >= kn) break;
+        const int32_t e = e0 - k;
+        const int32_t a = q4(va[u], k);
+        bool raw = false, war, waw;
+        if constexpr (OP == JP_OP_ADD_C) {
+          raw = earlier32(t.wA, q4(vb[u], k), lenA, e);
+          war = earlier32(t.rA, a, lenA, e);
+          waw = earlier32(t.wA, a, lenA, e);
+        } else if constexpr (OP == JP_OP_SAXPY) {
+          raw = earlier32(t.wA, a, lenA, e);
+          war = earlier32(t.rA, a, lenA, e);
+          waw = raw;
+        } else if constexpr (OP == JP_OP_PRIV_TMP) {
+          war = earlier32(rT, a, lenT, e);
+          waw = earlier32(t.wT, a, lenT, e) || earlier32(t.wA, q4(vb[u], k), lenA, e);
+        } else {
+          raw = earlier32(t.wA, q4(vb[u], k), lenA, e) || earlier32(t.wA, q4(vc[u], k), lenA, e);
+          war = earlier32(t.rA, a, lenA, e);
+          waw = earlier32(t.wA, a, lenA, e);
+        }
+        c_raw += raw; c_war += war; c_waw += waw;
+        if (raw && first == ~0ull) first = (unsigned long long)(L.base + (q << 2) + k);
+      }
     }
   }
+  c_raw = __reduce_add_sync(0xffffffffu, c_raw);
+  c_war = __reduce_add_sync(0xffffffffu, c_war);
+  c_waw = __reduce_add_sync(0xffffffffu, c_waw);
+  for (int o = 16; o; o >>= 1) {
+    const unsigned long long x = __shfl_xor_sync(0xffffffffu, first, o);
+    first = x < first ? x : first;
+  }
+  if ((threadIdx.x & 31) == 0) {
+    if (c_raw) atomicAdd(&s_cnt[0], (unsigned long long)c_raw);
+    if (c_war) atomicAdd(&s_cnt[1], (unsigned long long)c_war);
+    if (c_waw) atomicAdd(&s_cnt[2], (unsigned long long)c_waw);
+    if (first != ~0ull) atomicMin(&s_first, first);
+  }
+  JP_CTA_SYNC();
+  if (threadIdx.x < 3 && s_cnt[threadIdx.x]) atomicAdd((unsigned long long *)&hdr[H_RAW + threadIdx.x], s_cnt[threadIdx.x]);
+  if (threadIdx.x == 0 && s_first != ~0ull) atomicMin((unsigned long long *)&hdr[H_FIRST_RAW], s_first);
+}
+
+static int idx_vec(const DLoop &d) {
+  auto al = [](const int32_t *q) { return q == nullptr || ((uintptr_t)q & 15) == 0; };
+  return al(d.r) && al(d.w) && al(d.r2) && al(d.s);
 }
 
 // (bounds-guarded: classify may run before the host has seen the bad-index count)
@@ -105,44 +241,64 @@ __global__ void __launch_bounds__(256) k_prof_classify(DLoop L, Tabs t, uint32_t
   const int64_t warps = (int64_t)gridDim.x * (blockDim.x >> 5);
   unsigned long long c_raw = 0, c_war = 0, c_waw = 0, first = ~0ull;
   const int64_t tiles = (L.n + 31) >> 5;
-  for (int64_t tile = (int64_t)blockIdx.x * (blockDim.x >> 5) + (threadIdx.x >> 5); tile < tiles; tile += warps) {
-    const int64_t i = (tile << 5) + lane;
-    bool raw = false, war = false, waw = false;
-    if (i < L.n) {
-      const int32_t e = enc_gid(L.base + i);
-      if constexpr (OP == JP_OP_ADD_C) {
-        int64_t a = ixl(L, L.w, i);
-        raw = earlier(t.wA, ixl(L, L.r, i), L.lenA, e);
-        war = earlier(t.rA, a, L.lenA, e);
-        waw = earlier(t.wA, a, L.lenA, e);
-      } else if constexpr (OP == JP_OP_SAXPY) {
-        int64_t a = ixl(L, L.w, i);
-        raw = earlier(t.wA, a, L.lenA, e);
-        war = earlier(t.rA, a, L.lenA, e);
-        waw = raw;  // the same address is the exposed read and the write
-      } else if constexpr (OP == JP_OP_PRIV_TMP) {
-        int64_t a = ixl(L, L.s, i), b = ixl(L, L.w, i);
-        war = earlier(t.rT, a, L.lenT, e);
-        waw = earlier(t.wT, a, L.lenT, e) || earlier(t.wA, b, L.lenA, e);
-      } else {
-        int64_t a = ixl(L, L.w, i);
-        raw = earlier(t.wA, ixl(L, L.r, i), L.lenA, e) || earlier(t.wA, ixl(L, L.r2, i), L.lenA, e);
-        war = earlier(t.rA, a, L.lenA, e);
-        waw = earlier(t.wA, a, L.lenA, e);
+  // PRIV_TMP: minR(T) == minW(T) (every T write is also its covered read)
+  const int32_t *rT = OP == JP_OP_PRIV_TMP ? t.wT : t.rT;
+  // each warp takes kUnroll consecutive tiles per step; all loads before any use
+  for (int64_t tile0 = ((int64_t)blockIdx.x * (blockDim.x >> 5) + (threadIdx.x >> 5)) * kUnroll; tile0 < tiles;
+       tile0 += warps * kUnroll) {
+    int64_t ia[kUnroll], ib[kUnroll], ic[kUnroll];
+#pragma unroll
+    for (int u = 0; u < kUnroll; u++) {
+      const int64_t i = ((tile0 + u) << 5) + lane;
+      if (i < L.n) {
+        if constexpr (OP == JP_OP_ADD_C) { ia[u] = ixl(L, L.w, i); ib[u] = ixl(L, L.r, i); }
+        else if constexpr (OP == JP_OP_SAXPY) { ia[u] = ixl(L, L.w, i); }
+        else if constexpr (OP == JP_OP_PRIV_TMP) { ia[u] = ixl(L, L.s, i); ib[u] = ixl(L, L.w, i); }
+        else { ia[u] = ixl(L, L.w, i); ib[u] = ixl(L, L.r, i); ic[u] = ixl(L, L.r2, i); }
       }
     }
-    const unsigned bR = __ballot_sync(0xffffffffu, raw);
-    const unsigned bA = __ballot_sync(0xffffffffu, war);
-    const unsigned bW = __ballot_sync(0xffffffffu, waw);
-    if (lane == 0) {
-      c_raw += __popc(bR); c_war += __popc(bA); c_waw += __popc(bW);
-      if (raw_bits) raw_bits[tile] = bR;
-      if (bR && first == ~0ull) first = (unsigned long long)(L.base + (tile << 5) + __ffs(bR) - 1);
-      if (chunk_counts && (bR | bA | bW)) {
-        int64_t c = (tile << 5) / chunk;
-        if (bR) atomicAdd((unsigned long long *)&chunk_counts[3 * c + 0], (unsigned long long)__popc(bR));
-        if (bA) atomicAdd((unsigned long long *)&chunk_counts[3 * c + 1], (unsigned long long)__popc(bA));
-        if (bW) atomicAdd((unsigned long long *)&chunk_counts[3 * c + 2], (unsigned long long)__popc(bW));
+    bool raw[kUnroll], war[kUnroll], waw[kUnroll];
+#pragma unroll
+    for (int u = 0; u < kUnroll; u++) {   // table lookups, all issued before the ballots
+      const int64_t i = ((tile0 + u) << 5) + lane;
+      raw[u] = war[u] = waw[u] = false;
+      if (i < L.n) {
+        const int32_t e = enc_gid(L.base + i);
+        if constexpr (OP == JP_OP_ADD_C) {
+          raw[u] = earlier(t.wA, ib[u], L.lenA, e);
+          war[u] = earlier(t.rA, ia[u], L.lenA, e);
+          waw[u] = earlier(t.wA, ia[u], L.lenA, e);
+        } else if constexpr (OP == JP_OP_SAXPY) {
+          raw[u] = earlier(t.wA, ia[u], L.lenA, e);
+          war[u] = earlier(t.rA, ia[u], L.lenA, e);
+          waw[u] = raw[u];   // the same address is the exposed read and the write
+        } else if constexpr (OP == JP_OP_PRIV_TMP) {
+          war[u] = earlier(rT, ia[u], L.lenT, e);
+          waw[u] = earlier(t.wT, ia[u], L.lenT, e) || earlier(t.wA, ib[u], L.lenA, e);
+        } else {
+          raw[u] = earlier(t.wA, ib[u], L.lenA, e) || earlier(t.wA, ic[u], L.lenA, e);
+          war[u] = earlier(t.rA, ia[u], L.lenA, e);
+          waw[u] = earlier(t.wA, ia[u], L.lenA, e);
+        }
+      }
+    }
+#pragma unroll
+    for (int u = 0; u < kUnroll; u++) {
+      const int64_t tile = tile0 + u;
+      if (tile >= tiles) break;   // warp-uniform
+      const unsigned bR = __ballot_sync(0xffffffffu, raw[u]);
+      const unsigned bA = __ballot_sync(0xffffffffu, war[u]);
+      const unsigned bW = __ballot_sync(0xffffffffu, waw[u]);
+      if (lane == 0) {
+        c_raw += __popc(bR); c_war += __popc(bA); c_waw += __popc(bW);
+        if (raw_bits) raw_bits[tile] = bR;
+        if (bR && first == ~0ull) first = (unsigned long long)(L.base + (tile << 5) + __ffs(bR) - 1);
+        if (chunk_counts && (bR | bA | bW)) {
+          int64_t c = (tile << 5) / chunk;
+          if (bR) atomicAdd((unsigned long long *)&chunk_counts[3 * c + 0], (unsigned long long)__popc(bR));
+          if (bA) atomicAdd((unsigned long long *)&chunk_counts[3 * c + 1], (unsigned long long)__popc(bA));
+          if (bW) atomicAdd((unsigned long long *)&chunk_counts[3 * c + 2], (unsigned long long)__popc(bW));
+        }
       }
     }
   }
@@ -245,8 +401,9 @@ static int grid_for(int64_t n, int threads, int per_sm) {
 template <int OP, int DT>
 static void run_stamp(const DLoop &d, Tabs t, int64_t *hdr, size_t smem, cudaStream_t st) {
   (void)DT;
-  if (smem > 48 * 1024) cudaFuncSetAttribute(k_prof_stamp<OP>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-  k_prof_stamp<OP><<<grid_for(d.n, 256, 8), 256, smem, st>>>(d, t, hdr);
+  if (smem > 48 * 1024) cudaFuncSetAttribute(k_prof_stamp4<OP>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+  const int64_t nq = (d.n + 3) / 4;
+  k_prof_stamp4<OP><<<grid_for((nq + kQuadSteps - 1) / kQuadSteps, 256, 8), 256, smem, st>>>(d, t, idx_vec(d), hdr);
   note_launch();
 }
 
@@ -271,7 +428,7 @@ cudaError_t launch_prof_stamp(const Job &j, void *ws, const Layout &lo, cudaStre
   Tabs t = tabs_of(j.d, ws, lo);
   size_t smem = 0;
   if (t.sA) smem += (size_t)j.d.lenA * 4 * (t.rA ? 2 : 1);
-  if (t.sT) smem += (size_t)j.d.lenT * 4 * 2;
+  if (t.sT) smem += (size_t)j.d.lenT * 4;
   JP_DISPATCH(j.op, j.dt, run_stamp, j.d, t, hdr, smem, st);
   return launch_check();
 }
@@ -281,7 +438,12 @@ static void run_classify(const DLoop &d, Tabs t, uint32_t *bits, int64_t chunk, 
                          cudaStream_t st) {
   (void)DT;
   int64_t tiles = (d.n + 31) / 32;
-  k_prof_classify<OP><<<grid_for(tiles * 32, 256, 8), 256, 0, st>>>(d, t, bits, chunk, cc, hdr);
+  if (!bits && !cc) {
+    const int64_t nq = (d.n + 3) / 4;
+    k_prof_count4<OP><<<grid_for((nq + kQuadSteps - 1) / kQuadSteps, 256, 8), 256, 0, st>>>(d, t, idx_vec(d), hdr);
+  } else {
+    k_prof_classify<OP><<<grid_for((tiles + kUnroll - 1) / kUnroll * 32, 256, 8), 256, 0, st>>>(d, t, bits, chunk, cc, hdr);
+  }
   note_launch();
 }
 

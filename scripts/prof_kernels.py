@@ -37,6 +37,8 @@ if a.what in ("tls", "profile", "all"):
     ws = jp.workspace(L)
     for _ in range(a.reps):
         p = jp.jp_profile_density(L, ws)
-    jp.jp_run_tls(L, window=4096, w_max=4096, prof=p, ws=ws)
+    jp.jp_tls_guide(L, ws)
+    jp.jp_run_tls(L, window=4096, w_max=4096, path=3, prof=p, ws=ws, guided=True)   # k_tls_cluster
+    jp.jp_run_tls(L, window=0, w_max=4096, prof=p, ws=ws)                            # k_tls_cta (adaptive)
     torch.cuda.synchronize()
 print("done", jp.jp_launch_count())

@@ -10,6 +10,7 @@ import re
 import pytest
 import torch
 
+import oracle as O
 import oracle.sched as S
 import paper_conf_icpp_hanzlw13_b200 as jp
 from paper_conf_icpp_hanzlw13_b200 import _abi
@@ -186,3 +187,12 @@ def test_bad_arguments():
     with pytest.raises(jp.JPError) as e:
         jp.jp_ws_region(L, "header")
     assert e.value.status == _abi.JP_ERR_INDEX
+
+
+@pytest.mark.parametrize("n,raw", [(1 << 24, 16777), (1 << 24, 167772), (1 << 24, 1677722), (4096, 205), (100, 0),
+                                   (100, -1), (1000, 3), (7, 7), (1 << 20, 1)])
+def test_tls_first_window_matches_oracle(n, raw):
+    """The binding's host copy of reading A8's first window (used to label the
+    bench path) equals the oracle's definition."""
+    for w_max in (32, 4096, 65536):
+        assert jp.tls_first_window(n, raw, w_max) == O.tls_next_window(n, raw, -1, w_max)
