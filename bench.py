@@ -374,7 +374,9 @@ def run_jp(args):
                           "n_total": N2, "n_per_rank": s1 - s0, "partition": "task sharing, equal weights",
                           "l2": "inputs (3.2 GB) larger than L2 (126 MB); no flush needed",
                           "parallelism": f"iteration-range sharding x{world}"},
-               "roofline": {"bound": "hbm", "kernel": "k_doall_affine_vec<SAXPY,F32>", "achieved": achieved,
+               "roofline": {"bound": "hbm", "kernel": ["k_doall_affine_vec<SAXPY,F32>",
+                                                        "k_doall_affine_tma<SAXPY,F32>"][jp.jp_doall_kernel(-1)],
+                            "achieved": achieved,
                             "peak": hbm, "unit": "GB/s", "frac": achieved / hbm, "traffic": traffic,
                             "algorithmic_bytes_per_iter": BYTES_PER_ITER_SAXPY, "peak_source": peak_src,
                             "kernel_ms": kernel_ms},

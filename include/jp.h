@@ -184,6 +184,12 @@ int32_t jp_select_mode(const jp_loop *L /* host */, const jp_profile *p /* host,
  * nullable) that shows any dependence: JP_ERR_ILLEGAL_MODE.  Without a profile
  * the caller asserts legality.  If index arrays are present and p == NULL the
  * indices are validated first (syncs).                                        */
+/* Kernel of the affine (all-NULL-index) DOALL body, process-wide: 0 = 16-byte
+ * LDG/STG grid-stride stream, 1 = bulk-copy (TMA) staged ring through shared
+ * memory (default).  which = 0 or 1 sets it; any other value only queries.
+ * Returns the current choice.  Both are bit-exact; DESIGN.md Sec.6 has the
+ * measured comparison (initial value from env JP_DOALL_KERNEL).            */
+int32_t jp_doall_kernel(int32_t which);
 jp_status jp_run_doall(const jp_loop *L, const jp_profile *p, void *ws, size_t ws_bytes,
                        jp_stream_t st);
 

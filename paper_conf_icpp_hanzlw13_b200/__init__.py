@@ -23,7 +23,7 @@ from ._abi import (  # noqa: F401
 __all__ = [
     "Loop", "workspace", "jp_workspace_bytes", "jp_ws_region", "jp_validate", "jp_profile_stamp",
     "jp_profile_classify", "jp_profile_density", "jp_select_mode", "jp_run_doall", "jp_run_privatized",
-    "jp_priv_stream", "jp_priv_finalize", "jp_tls_guide", "tls_first_window", "jp_run_tls", "jp_schedule", "jp_stage_bytes", "jp_schedule_host",
+    "jp_priv_stream", "jp_priv_finalize", "jp_doall_kernel", "jp_tls_guide", "tls_first_window", "jp_run_tls", "jp_schedule", "jp_stage_bytes", "jp_schedule_host",
     "jp_plan_sharing", "jp_plan_stealing", "jp_merge_apply", "jp_last_error", "jp_version", "jp_launch_count",
 ]
 
@@ -191,6 +191,11 @@ def jp_priv_stream(loop: Loop, prof=None, ws=None, clear_keys=True, stream=None)
 def jp_priv_finalize(loop: Loop, ws, stream=None):
     p, nb = _ws(ws)
     check(lib().jp_priv_finalize(loop.ref, p, nb, _stream(stream)))
+
+
+def jp_doall_kernel(which: int = -1) -> int:
+    """Affine DOALL kernel choice: 0 LDG/STG.128 stream, 1 bulk-copy (TMA) staged; -1 queries."""
+    return int(lib().jp_doall_kernel(int(which)))
 
 
 def tls_first_window(n: int, raw_iters: int, w_max: int = 4096) -> int:

@@ -83,6 +83,7 @@ SIGNATURES = [
     ("jp_run_privatized", _I32, [_P(jp_loop), _P(jp_profile), _V, _SZ, _V]),
     ("jp_priv_stream", _I32, [_P(jp_loop), _P(jp_profile), _V, _SZ, _I32, _V]),
     ("jp_priv_finalize", _I32, [_P(jp_loop), _V, _SZ, _V]),
+    ("jp_doall_kernel", _I32, [_I32]),
     ("jp_tls_guide", _I32, [_P(jp_loop), _V, _SZ, _V]),
     ("jp_run_tls", _I32, [_P(jp_loop), _P(jp_tls_cfg), _P(jp_profile), _V, _SZ, _P(jp_tls_stats), _V]),
     ("jp_schedule", _I32, [_P(jp_loop), _P(jp_sched_cfg), _V, _SZ, _P(jp_sched_result), _V]),

@@ -244,6 +244,11 @@ const char *jp_last_error(void) { return g_err.c_str(); }
 const char *jp_version(void) { return "jp-b200 0.1 (sm_100a)"; }
 int64_t jp_launch_count(void) { return g_launches.load(); }
 
+int32_t jp_doall_kernel(int32_t which) {
+  if (which == 0 || which == 1) set_doall_kernel_choice(which);
+  return doall_kernel_choice();
+}
+
 size_t jp_workspace_bytes(const jp_loop *L, int32_t uses) {
   if (!L || check_loop(L) == JP_ERR_ARG) return 0;
   return layout_end(layout(L), uses);

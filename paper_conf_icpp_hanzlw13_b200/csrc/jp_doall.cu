@@ -9,6 +9,8 @@
 //   multiple of the SM count.  12 B/iteration for SAXPY (X 4 + Y 4 read, Y 4 written).
 // k_doall_generic: indirect bodies (config 1 at 0%, the config-5 head):
 //   coalesced index streams, gathered/scattered element accesses.
+#include <atomic>
+#include <cstdlib>
 #include "jp_host.h"
 
 namespace jp {
@@ -68,6 +70,108 @@ __global__ void __launch_bounds__(kAffThreads) k_doall_affine_vec(DLoop L, int64
   }
 }
 
+// k_doall_affine_tma: the same affine loop staged through shared memory with
+// bulk copies (cp.async.bulk, the TMA engine's 1-D mode): one CTA per SM, a
+// kTmaStages-deep ring of 16 KiB tiles per stream, mbarrier completion for the
+// loads (one elected thread arms expect_tx and issues both copies), the body
+// computed in place in shared memory by all threads, then one bulk store per
+// tile (bulk_group; a stage is reloaded once its store has finished reading).
+// Measured against k_doall_affine_vec in DESIGN.md Sec.6 (the faster one is
+// the default).
+constexpr int kTmaTile = 4096;                 // elements per tile per stream (16 KiB)
+constexpr int kTmaStages = 4;
+constexpr int kTmaThreads = 256;
+
+__device__ __forceinline__ uint32_t smem_u32(const void *p) { return (uint32_t)__cvta_generic_to_shared(p); }
+__device__ __forceinline__ void mbar_init(unsigned long long *b, uint32_t count) {
+  asm volatile("mbarrier.init.shared::cta.b64 [%0], %1;" ::"r"(smem_u32(b)), "r"(count) : "memory");
+}
+__device__ __forceinline__ void mbar_expect_tx(unsigned long long *b, uint32_t bytes) {
+  asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(smem_u32(b)), "r"(bytes) : "memory");
+}
+__device__ __forceinline__ void mbar_wait(unsigned long long *b, uint32_t parity) {
+  asm volatile(
+      "{\n\t.reg .pred p;\n"
+      "WAIT_%=:\n\t"
+      "mbarrier.try_wait.parity.shared::cta.b64 p, [%0], %1;\n\t"
+      "@!p bra WAIT_%=;\n\t}" ::"r"(smem_u32(b)), "r"(parity) : "memory");
+}
+__device__ __forceinline__ void bulk_load(void *dst, const void *src, uint32_t bytes, unsigned long long *bar) {
+  asm volatile("cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];"
+               ::"r"(smem_u32(dst)), "l"(src), "r"(bytes), "r"(smem_u32(bar)) : "memory");
+}
+__device__ __forceinline__ void bulk_store(void *dst, const void *src, uint32_t bytes) {
+  asm volatile("cp.async.bulk.global.shared::cta.bulk_group [%0], [%1], %2;" ::"l"(dst), "r"(smem_u32(src)), "r"(bytes)
+               : "memory");
+}
+
+template <int OP, int DT>
+__global__ void __launch_bounds__(kTmaThreads, 1) k_doall_affine_tma(DLoop L, int64_t ntiles) {
+  constexpr bool readsA = OP != JP_OP_PRIV_TMP;
+  constexpr bool readsX = OP == JP_OP_SAXPY || OP == JP_OP_PRIV_TMP;
+  constexpr int NB = 2;   // buffers per stage: A (in/out) and X (PRIV_TMP: T out, X in)
+  extern __shared__ __align__(128) uint32_t tsm[];   // [stage][NB][kTmaTile]
+  __shared__ __align__(8) unsigned long long full[kTmaStages];
+  const int tid = threadIdx.x;
+  const uint32_t bytes_in = (uint32_t)(((readsA ? 1 : 0) + (readsX ? 1 : 0)) * kTmaTile * 4);
+  // this CTA's tiles: t = blockIdx.x + k * gridDim.x
+  const int64_t my = ntiles > blockIdx.x ? (ntiles - 1 - blockIdx.x) / gridDim.x + 1 : 0;
+  auto tile_of = [&](int64_t k) { return (int64_t)blockIdx.x + k * gridDim.x; };
+  auto issue = [&](int64_t k) {
+    const int s = (int)(k % kTmaStages);
+    const int64_t e0 = tile_of(k) * kTmaTile;
+    uint32_t *bA = tsm + (size_t)s * NB * kTmaTile, *bX = bA + kTmaTile;
+    mbar_expect_tx(&full[s], bytes_in);
+    if constexpr (readsA) bulk_load(bA, L.A + e0, kTmaTile * 4, &full[s]);
+    if constexpr (readsX) bulk_load(bX, L.X + e0, kTmaTile * 4, &full[s]);
+  };
+  if (tid == 0) {
+    for (int s = 0; s < kTmaStages; s++) mbar_init(&full[s], 1);
+    asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+  }
+  __syncthreads();
+  if (tid == 0)
+    for (int64_t k = 0; k < kTmaStages - 1 && k < my; k++) issue(k);
+  for (int64_t k = 0; k < my; k++) {
+    const int s = (int)(k % kTmaStages);
+    const uint32_t parity = (uint32_t)((k / kTmaStages) & 1);
+    uint32_t *bA = tsm + (size_t)s * NB * kTmaTile, *bX = bA + kTmaTile;
+    mbar_wait(&full[s], parity);
+    uint4 *A4 = reinterpret_cast<uint4 *>(bA);
+    uint4 *X4 = reinterpret_cast<uint4 *>(bX);
+#pragma unroll
+    for (int v = tid; v < kTmaTile / 4; v += kTmaThreads) {
+      uint4 a = readsA ? A4[v] : make_uint4(0, 0, 0, 0), x = readsX ? X4[v] : make_uint4(0, 0, 0, 0), t;
+      vec_body<OP, DT>(x, a, t, L.c0, L.c1);
+      A4[v] = a;
+      if constexpr (OP == JP_OP_PRIV_TMP) X4[v] = t;   // X is consumed: its buffer carries T out
+    }
+    asm volatile("fence.proxy.async.shared::cta;" ::: "memory");   // generic writes -> async proxy
+    __syncthreads();
+    if (tid == 0) {
+      const int64_t e0 = tile_of(k) * kTmaTile;
+      bulk_store(L.A + e0, bA, kTmaTile * 4);
+      if constexpr (OP == JP_OP_PRIV_TMP) bulk_store(L.T + e0, bX, kTmaTile * 4);
+      asm volatile("cp.async.bulk.commit_group;" ::: "memory");
+      // refill the stage used one iteration ago once its store has read smem
+      if (k + kTmaStages - 1 < my) {
+        asm volatile("cp.async.bulk.wait_group.read 1;" ::: "memory");
+        issue(k + kTmaStages - 1);
+      }
+    }
+  }
+  if (tid == 0) asm volatile("cp.async.bulk.wait_group 0;" ::: "memory");
+  // element tail [ntiles * kTmaTile, n): CTA 0, plain accesses
+  if (blockIdx.x == 0) {
+    for (int64_t i = ntiles * kTmaTile + tid; i < L.n; i += kTmaThreads) {
+      uint32_t va = 0, vt = 0;
+      body_values<OP, DT>(L, i, L.A, va, vt);
+      if constexpr (OP == JP_OP_PRIV_TMP) L.T[i] = vt;
+      L.A[i] = va;
+    }
+  }
+}
+
 template <int OP, int DT>
 __global__ void __launch_bounds__(256) k_doall_generic(DLoop L) {
   const int64_t stride = (int64_t)gridDim.x * blockDim.x;
@@ -81,11 +185,33 @@ __global__ void __launch_bounds__(256) k_doall_generic(DLoop L) {
 
 static bool aligned16(const void *p) { return ((uintptr_t)p & 15) == 0; }
 
+// affine DOALL kernel choice (jp_doall_kernel): 0 LDG/STG.128 grid-stride, 1 bulk-copy (TMA) staged
+// (default: config 2 measured 6.48 vs 6.25 TB/s)
+static std::atomic<int> g_doall_kernel{-1};
+int doall_kernel_choice() {
+  int v = g_doall_kernel.load();
+  if (v < 0) {
+    const char *e = getenv("JP_DOALL_KERNEL");   // default: bulk-copy staged (measured faster)
+    v = e && e[0] == '0' ? 0 : 1;
+    g_doall_kernel.store(v);
+  }
+  return v;
+}
+void set_doall_kernel_choice(int v) { g_doall_kernel.store(v); }
+
 template <int OP, int DT>
 static void run_doall(const DLoop &d, cudaStream_t st, int max_ctas) {
   const bool affine = !d.r && !d.r2 && !d.w && !d.s && d.ioff == 0;
   int sms = num_sms();
-  if (affine && aligned16(d.A) && (!d.X || aligned16(d.X)) && (!d.T || aligned16(d.T))) {
+  if (doall_kernel_choice() == 1 && affine && aligned16(d.A) && (!d.X || aligned16(d.X)) && (!d.T || aligned16(d.T))) {
+    const int64_t ntiles = d.n / kTmaTile;
+    const size_t smem = (size_t)kTmaStages * 2 * kTmaTile * 4;
+    cudaFuncSetAttribute(k_doall_affine_tma<OP, DT>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+    int64_t cap = sms;
+    if (max_ctas > 0 && cap > max_ctas) cap = max_ctas;
+    const int grid = (int)(ntiles < 1 ? 1 : ntiles < cap ? ntiles : cap);
+    k_doall_affine_tma<OP, DT><<<grid, kTmaThreads, smem, st>>>(d, ntiles);
+  } else if (affine && aligned16(d.A) && (!d.X || aligned16(d.X)) && (!d.T || aligned16(d.T))) {
     int64_t nvec = d.n / 4;
     int64_t need = (nvec + kAffThreads * kAffUnroll - 1) / (kAffThreads * kAffUnroll);
     int64_t cap = (int64_t)sms * 8;

@@ -51,6 +51,8 @@ cudaError_t launch_prof_stamp(const Job &j, void *ws, const Layout &lo, cudaStre
 cudaError_t launch_prof_classify(const Job &j, void *ws, const Layout &lo, uint32_t *raw_bits,
                                  int64_t chunk, int64_t *chunk_counts, cudaStream_t st);
 cudaError_t launch_doall(const Job &j, cudaStream_t st, int max_ctas = 0);
+int doall_kernel_choice();
+void set_doall_kernel_choice(int v);
 cudaError_t launch_priv_stream(const Job &j, void *ws, const Layout &lo, bool clear_keys,
                                cudaStream_t st, int max_ctas = 0);
 cudaError_t launch_priv_finalize(const Job &j, void *ws, const Layout &lo, cudaStream_t st);

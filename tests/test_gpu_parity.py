@@ -170,9 +170,18 @@ def test_illegal_modes_and_workspace():
 # ---------------------------------------------------------------------------
 # DOALL
 # ---------------------------------------------------------------------------
+@pytest.fixture(params=[0, 1], ids=["ldg128", "tma"])
+def doall_kernel(request):
+    """Both affine DOALL kernels (jp_doall_kernel): LDG/STG.128 stream and bulk-copy staged."""
+    old = jp.jp_doall_kernel(-1)
+    jp.jp_doall_kernel(request.param)
+    yield request.param
+    jp.jp_doall_kernel(old)
+
+
 @pytest.mark.parametrize("op,dt", list(itertools.product(OPS, DTS)))
-def test_doall_affine(op, dt):
-    n = (1 << 20) + 3
+@pytest.mark.parametrize("n", [(1 << 20) + 3, 4096 * 5, 100, 4096 * 149 + 17])
+def test_doall_affine(op, dt, n, doall_kernel):
     wl = random_loop(77 + op * 2 + dt, op, dt, n, null_prob=1.0)   # all indices NULL
     _, A, T = O.run_seq(to_oracle(wl))
     g = gpu(wl)
@@ -219,7 +228,7 @@ def test_doall_indirect_permutation(op, dt):
     check_arrays(g, A, T)
 
 
-def test_config2_full_size_sampled():
+def test_config2_full_size_sampled(doall_kernel):
     """BASELINE size N=2^28 in the bench's launch configuration; outputs sampled
     and recomputed one by one by the oracle."""
     n = 1 << 28
