@@ -138,6 +138,87 @@ __global__ void __launch_bounds__(kPrivThreads) k_priv_tmp_vec(DLoop L, unsigned
   }
 }
 
+// Same loop, bulk-copy (TMA) staged: one CTA per SM walks its tiles in
+// DESCENDING order through a kPrivStages ring of {X, s} 16 KiB tiles (mbarrier
+// completion), computes Y in place of X in shared memory and bulk-stores it;
+// the slot table is updated from the staged s tile (descending inside the tile
+// too, so the check-before-atomic filter keeps working).
+constexpr int kPrivTile = 4096, kPrivStages = 4, kPrivTmaThreads = 256;
+
+template <int DT>
+__global__ void __launch_bounds__(kPrivTmaThreads, 1) k_priv_tmp_tma(DLoop L, unsigned long long *kT, int64_t ntiles) {
+  extern __shared__ __align__(128) uint32_t psm[];   // [stage][2][tile] then tT[lenT]
+  __shared__ __align__(8) unsigned long long full[kPrivStages];
+  uint32_t *tT = psm + (size_t)kPrivStages * 2 * kPrivTile;
+  const int tid = threadIdx.x;
+  for (int64_t k = tid; k < L.lenT; k += kPrivTmaThreads) tT[k] = 0;
+  // this CTA's tiles, highest first: t = ntiles-1-blockIdx.x - k*gridDim.x
+  const int64_t my = ntiles > blockIdx.x ? (ntiles - 1 - blockIdx.x) / gridDim.x + 1 : 0;
+  auto tile_of = [&](int64_t k) { return ntiles - 1 - (int64_t)blockIdx.x - k * gridDim.x; };
+  auto issue = [&](int64_t k) {
+    const int sg = (int)(k % kPrivStages);
+    const int64_t e0 = tile_of(k) * kPrivTile;
+    uint32_t *bX = psm + (size_t)sg * 2 * kPrivTile, *bS = bX + kPrivTile;
+    mbar_expect_tx(&full[sg], 2 * kPrivTile * 4);
+    bulk_load(bX, L.X + e0, kPrivTile * 4, &full[sg]);
+    bulk_load(bS, L.s + e0, kPrivTile * 4, &full[sg]);
+  };
+  if (tid == 0) {
+    for (int sg = 0; sg < kPrivStages; sg++) mbar_init(&full[sg], 1);
+    asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+  }
+  __syncthreads();
+  if (tid == 0)
+    for (int64_t k = 0; k < kPrivStages - 1 && k < my; k++) issue(k);
+  for (int64_t k = 0; k < my; k++) {
+    const int sg = (int)(k % kPrivStages);
+    uint32_t *bX = psm + (size_t)sg * 2 * kPrivTile, *bS = bX + kPrivTile;
+    mbar_wait(&full[sg], (uint32_t)((k / kPrivStages) & 1));
+    const int64_t e0 = tile_of(k) * kPrivTile;
+    uint4 *X4 = reinterpret_cast<uint4 *>(bX);
+    const int4 *S4 = reinterpret_cast<const int4 *>(bS);
+#pragma unroll
+    for (int q = 0; q < kPrivTile / 4 / kPrivTmaThreads; q++) {
+      const int v = kPrivTile / 4 - 1 - (q * kPrivTmaThreads + tid);   // descending in the tile
+      const uint4 x = X4[v];
+      const int4 sv = S4[v];
+      uint4 y;
+      y.x = op_add<DT>(op_mul<DT>(L.c0, x.x), L.c1);
+      y.y = op_add<DT>(op_mul<DT>(L.c0, x.y), L.c1);
+      y.z = op_add<DT>(op_mul<DT>(L.c0, x.z), L.c1);
+      y.w = op_add<DT>(op_mul<DT>(L.c0, x.w), L.c1);
+      X4[v] = y;
+      const int64_t i0 = e0 + 4 * v;
+      smem_last(tT, sv.w, i0 + 3);
+      smem_last(tT, sv.z, i0 + 2);
+      smem_last(tT, sv.y, i0 + 1);
+      smem_last(tT, sv.x, i0 + 0);
+    }
+    asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
+    __syncthreads();
+    if (tid == 0) {
+      bulk_store(L.A + e0, bX, kPrivTile * 4);
+      asm volatile("cp.async.bulk.commit_group;" ::: "memory");
+      if (k + kPrivStages - 1 < my) {
+        asm volatile("cp.async.bulk.wait_group.read 1;" ::: "memory");
+        issue(k + kPrivStages - 1);
+      }
+    }
+  }
+  if (tid == 0) asm volatile("cp.async.bulk.wait_group 0;" ::: "memory");
+  if (blockIdx.x == 0) {   // element tail [ntiles * tile, n)
+    for (int64_t i = ntiles * kPrivTile + tid; i < L.n; i += kPrivTmaThreads) {
+      L.A[i] = op_add<DT>(op_mul<DT>(L.c0, L.X[i]), L.c1);
+      smem_last(tT, L.s[i], i);
+    }
+  }
+  __syncthreads();
+  for (int64_t b = tid; b < L.lenT; b += kPrivTmaThreads) {
+    const uint32_t e = tT[b];
+    if (e) atomicMax(&kT[b], pack_key(L.base + e - 1, op_mul<DT>(L.c0, L.X[e - 1])));
+  }
+}
+
 __global__ void k_apply_keys(uint32_t *arr, int64_t len, const unsigned long long *keys) {
   const int64_t stride = (int64_t)gridDim.x * blockDim.x;
   for (int64_t a = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; a < len; a += stride) {
@@ -155,6 +236,17 @@ static void run_priv(const DLoop &d, unsigned long long *kA, unsigned long long 
   if constexpr (OP == JP_OP_PRIV_TMP) {
     if (!d.r && !d.w && d.s && d.ioff == 0 && kT && !kA && d.lenT <= kSmemSlots && al16(d.X) && al16(d.s) &&
         al16(d.A)) {
+      if (doall_kernel_choice() == 1) {   // bulk-copy staged (the DOALL kernel choice covers both streams)
+        const int64_t ntiles = d.n / kPrivTile;
+        const size_t smem = (size_t)kPrivStages * 2 * kPrivTile * 4 + (size_t)d.lenT * 4;
+        cudaFuncSetAttribute(k_priv_tmp_tma<DT>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+        int g = num_sms();
+        if (max_ctas > 0 && g > max_ctas) g = max_ctas;
+        if (ntiles < g) g = (int)(ntiles < 1 ? 1 : ntiles);
+        k_priv_tmp_tma<DT><<<g, kPrivTmaThreads, smem, st>>>(d, kT, ntiles);
+        note_launch();
+        return;
+      }
       int64_t nvec = d.n / 4;
       int64_t need = (nvec + kPrivThreads * 2 - 1) / (kPrivThreads * 2);
       if (need < grid) grid = (int)(need < 1 ? 1 : need);

@@ -246,8 +246,8 @@ def test_config2_full_size_sampled(doall_kernel):
 # ---------------------------------------------------------------------------
 # privatized
 # ---------------------------------------------------------------------------
-@pytest.mark.parametrize("n", [1, 31, 4096 + 7, (1 << 20) + 5])
-def test_priv_config4(n):
+@pytest.mark.parametrize("n", [1, 31, 4096 + 7, 4096 * 3, (1 << 20) + 5, 4096 * 300 + 4099])
+def test_priv_config4(n, doall_kernel):
     wl = synth.config4(n=n)
     ref = to_oracle(wl)
     _, A, T = O.run_seq(ref)
@@ -315,7 +315,7 @@ def test_priv_split_merge_equals_whole():
     check_arrays(g, A, T)
 
 
-def test_config4_full_size():
+def test_config4_full_size(doall_kernel):
     """BASELINE size N=2^26 (bench launch configuration), compared in full."""
     wl = synth.config4()
     _, A, T = O.run_seq(to_oracle(wl))
