@@ -28,6 +28,7 @@ constexpr int kSmemSlots = 4096;          // arrays this small are pre-aggregate
 constexpr int kTlsCtaThreads = JP_TLS_THREADS;   // single-CTA TLS path
 constexpr int kTlsCtaIpt = JP_TLS_IPT;           // -> W <= 4096
 constexpr int kTlsCtaWmax = kTlsCtaThreads * kTlsCtaIpt;
+constexpr int kTlsFillThreads = 128;             // threads that issue the index-ring copies
 constexpr int kTlsHashLog = JP_TLS_HASHLOG;      // 8192 slots = 2 x W_max
 constexpr int kTlsHash = 1 << kTlsHashLog;
 constexpr int kTlsGridThreads = 512;

@@ -76,6 +76,12 @@ __host__ __device__ inline int64_t next_window(int64_t n, int64_t prof_raw, int6
   }
   return clamp64(pow2ceil64(2 * (prev > 16 ? prev : 16)), 32, w_max);
 }
+// the step rule alone (device, 32-bit, no division): clamp(pow2ceil(2*max(c,16)), 32, w_max)
+__device__ __forceinline__ int next_window_step(int prev, int w_max) {
+  const unsigned x = 2u * (unsigned)(prev > 16 ? prev : 16);
+  const int p = (int)(1u << (32 - __clz(x - 1)));
+  return p < 32 ? 32 : p > w_max ? w_max : p;
+}
 int64_t tls_next_window(int64_t n, int64_t prof_raw, int64_t prev, int64_t w_max) {
   return next_window(n, prof_raw, prev, w_max);
 }
@@ -176,32 +182,41 @@ __global__ void __launch_bounds__(kTlsCtaThreads, 1)
 
   // ring fill up to [ws_, ws_ + RL): index chunks of 4 (16-byte copies when
   // aligned; hi % 4 == 0 or hi == n) and guide words [ws_/32, ws_/32 + RB)
-  int64_t hi = 0, bhi = 0;
-  auto fill = [&](int64_t ws_) {
-    int64_t to = (ws_ + RL) & ~(int64_t)3;
-    if (to > L.n) to = L.n;
-    if (to > hi) {
-      const int64_t c0 = hi >> 2, c1 = (to + 3) >> 2;
-      for (int64_t c = c0 + tid; c < c1; c += T) {
-        const int64_t i0 = c << 2;
+  // (32-bit positions: n <= 2^31 - 2 and ws + RL < 2^32)
+  const uint32_t n32 = (uint32_t)L.n;
+  const bool s0 = src[0] != nullptr, s1 = src[1] != nullptr, s2 = src[2] != nullptr;
+  uint32_t hi = 0, bhi = 0;
+  auto fill = [&](uint32_t ws_) {
+    uint32_t to = (ws_ + (uint32_t)RL) & ~3u;
+    if (to > n32) to = n32;
+    if (tid < kTlsFillThreads && to > hi) {   // a few warps issue the copies; the rest skip
+      const uint32_t c1 = (to + 3) >> 2;
+      for (uint32_t c = (hi >> 2) + tid; c < c1; c += kTlsFillThreads) {
+        const uint32_t i0 = c << 2;
         const int slot = (int)(i0 & (RL - 1));
-#pragma unroll
-        for (int q = 0; q < NS; q++) {
-          if (!src[q]) continue;
-          if (R.al16 && i0 + 4 <= L.n) cp_async16(&ring[q * RL + slot], src[q] + i0);
-          else
-            for (int e = 0; e < 4; e++)
-              if (i0 + e < L.n) cp_async4(&ring[q * RL + slot + e], src[q] + i0 + e);
+        if (R.al16 && i0 + 4 <= n32) {
+          if (s0) cp_async16(&ring[slot], src[0] + i0);
+          if (s1) cp_async16(&ring[RL + slot], src[1] + i0);
+          if constexpr (NS == 3) if (s2) cp_async16(&ring[2 * RL + slot], src[2] + i0);
+        } else {
+          for (uint32_t e = 0; e < 4; e++) {
+            if (i0 + e >= n32) break;
+            if (s0) cp_async4(&ring[slot + e], src[0] + i0 + e);
+            if (s1) cp_async4(&ring[RL + slot + e], src[1] + i0 + e);
+            if constexpr (NS == 3) if (s2) cp_async4(&ring[2 * RL + slot + e], src[2] + i0 + e);
+          }
         }
       }
-      hi = to;
     }
+    if (to > hi) hi = to;
     if constexpr (GUIDED) {
-      const int64_t bto = (ws_ >> 5) + RB < nwords ? (ws_ >> 5) + RB : nwords;
-      for (int64_t g = bhi + tid; g < bto; g += T) {
-        cp_async4(&bring[g & (RB - 1)], gbits + g);
-        cp_async4(&bring[RB + (g & (RB - 1))], gbits + nwords + g);
-      }
+      uint32_t bto = (ws_ >> 5) + (uint32_t)RB;
+      if (bto > (uint32_t)nwords) bto = (uint32_t)nwords;
+      if (tid < kTlsFillThreads)
+        for (uint32_t g = bhi + tid; g < bto; g += kTlsFillThreads) {
+          cp_async4(&bring[g & (RB - 1)], gbits + g);
+          cp_async4(&bring[RB + (g & (RB - 1))], gbits + nwords + g);
+        }
       if (bto > bhi) bhi = bto;
     }
     cp_async_commit();
@@ -212,19 +227,20 @@ __global__ void __launch_bounds__(kTlsCtaThreads, 1)
 
   const bool dc = n_exposed<OP>() > 0 && P.hashA;
   const bool insA = P.hashA && (WAW || dc);   // A keys: commit order (WAW) and/or conflict detection
-  int64_t ws = 0;
-  int64_t W = P.window > 0 ? P.window : next_window(L.n, P.prof_raw, -1, P.w_max);
+  uint32_t ws = 0;
+  int W = (int)(P.window > 0 ? P.window : next_window(L.n, P.prof_raw, -1, P.w_max));
+  const int wfix = (int)P.window, wmax = (int)P.w_max;
   long long committed = 0, executed = 0, windows = 0, viol = 0;
   int par = 0;
 #ifdef JP_TLS_TRACE
   const bool trc = tid == 0;
 #endif
-  while (ws < L.n) {
+  while (ws < n32) {
 #ifdef JP_TLS_TRACE
     const bool tr = trc && windows < kTraceWin;
 #endif
     TLS_TR(0);
-    const int span = (int)(W < L.n - ws ? W : L.n - ws);
+    const int span = (int)((uint32_t)W < n32 - ws ? (uint32_t)W : n32 - ws);
     if (tid == 0) s_fv[par ^ 1] = INT32_MAX;
     fill(ws);   // reuses the slots of iterations < ws
     TLS_TR(8);
@@ -240,11 +256,12 @@ __global__ void __launch_bounds__(kTlsCtaThreads, 1)
       rawk[k] = true;
       slA[k] = slT[k] = -1;
       if (off < span) {
-        const int64_t i = ws + off;
+        const uint32_t i = ws + (uint32_t)off;
         const int slot = (int)(i & (RL - 1));
-        ix0[k] = src[0] ? ring[slot] : (int32_t)(L.ioff + i);
-        ix1[k] = src[1] ? ring[RL + slot] : (int32_t)(L.ioff + i);
-        if constexpr (NS == 3) ix2[k] = src[2] ? ring[2 * RL + slot] : (int32_t)(L.ioff + i);
+        const int32_t id = (int32_t)L.ioff + (int32_t)i;
+        ix0[k] = s0 ? ring[slot] : id;
+        ix1[k] = s1 ? ring[RL + slot] : id;
+        if constexpr (NS == 3) ix2[k] = s2 ? ring[2 * RL + slot] : id;
       }
     }
     TLS_TR(9);
@@ -269,7 +286,7 @@ __global__ void __launch_bounds__(kTlsCtaThreads, 1)
       if (off < span) {
         bool ins = insA;
         if constexpr (GUIDED) {
-          const int64_t i = ws + off;
+          const uint32_t i = ws + (uint32_t)off;
           const int b = (int)((i >> 5) & (RB - 1)), sh = (int)(i & 31);
           rawk[k] = (bring[b] >> sh) & 1u;
           ins = ins && ((bring[RB + b] >> sh) & 1u);
@@ -358,8 +375,8 @@ __global__ void __launch_bounds__(kTlsCtaThreads, 1)
     TLS_SYNC();   // commits and prefetched indices visible to the next SE, hash clean
     TLS_TR(7);
     committed += fv; executed += span; windows++; viol += fv < span;
-    ws += fv;
-    W = P.window > 0 ? P.window : next_window(L.n, P.prof_raw, fv, P.w_max);
+    ws += (uint32_t)fv;
+    W = wfix > 0 ? wfix : next_window_step(fv, wmax);
     par ^= 1;
     TLS_TR(13);
   }
