@@ -587,42 +587,56 @@ __global__ void __launch_bounds__(kTlsClThreads, 1)
   const int64_t qmax = (ngroups - crank + C - 1) >> logC;   // groups owned by this CTA
 
   // ring refill: this CTA's groups g = q*C + crank for q in [q_fill, q_to);
-  // one commit group per call (possibly empty) for the wait_group accounting
-  int64_t q_fill = 0;
-  auto refill = [&](int64_t ws_) {
-    int64_t q_to = ((ws_ >> 5) >> logC) + RG;
-    if (q_to > qmax) q_to = qmax;
-    const int nq = (int)(q_to - q_fill);
-    if (nq > 0) {
+  // issued by the first kTlsFillThreads threads; one commit group per call
+  // (possibly empty) for the wait_group accounting.  32-bit positions:
+  // n <= 2^31 - 2, so group and q counts fit.
+  const uint32_t n32 = (uint32_t)L.n;
+  const bool s0 = src[0] != nullptr, s1 = src[1] != nullptr, s2 = src[2] != nullptr;
+  uint32_t q_fill = 0;
+  auto refill = [&](uint32_t ws_) {
+    uint32_t q_to = ((ws_ >> 5) >> logC) + (uint32_t)RG;
+    if (q_to > (uint32_t)qmax) q_to = (uint32_t)qmax;
+    if (tid < kTlsFillThreads && q_to > q_fill) {
+      const uint32_t nq = q_to - q_fill;
       if (R.al16) {
-        for (int u = tid; u < nq * NS * 8; u += kTlsClThreads) {   // 8 x 16 B per (group, stream)
-          const int qq = u / (NS * 8), rem = u - qq * (NS * 8), s = rem >> 3, part = rem & 7;
-          if (!src[s]) continue;
-          const int64_t q = q_fill + qq;
-          const int64_t i0 = (((q << logC) + crank) << 5) + part * 4;
-          int32_t *dst = &ring[(s * RG + (int)(q & (RG - 1))) * 32 + part * 4];
-          if (i0 + 4 <= L.n) cp_async16(dst, src[s] + i0);
-          else
-            for (int e = 0; e < 4; e++) if (i0 + e < L.n) cp_async4(dst + e, src[s] + i0 + e);
+        for (uint32_t u = tid; u < nq * 8; u += kTlsFillThreads) {   // 8 x 16 B per group and stream
+          const uint32_t q = q_fill + (u >> 3), part = u & 7;
+          const uint32_t i0 = (((q << logC) + (uint32_t)crank) << 5) + part * 4;
+          const int d = (int)(q & (RG - 1)) * 32 + (int)part * 4;
+          if (i0 + 4 <= n32) {
+            if (s0) cp_async16(&ring[d], src[0] + i0);
+            if (s1) cp_async16(&ring[RG * 32 + d], src[1] + i0);
+            if constexpr (NS == 3) if (s2) cp_async16(&ring[2 * RG * 32 + d], src[2] + i0);
+          } else {
+            for (uint32_t e = 0; e < 4; e++) {
+              if (i0 + e >= n32) break;
+              if (s0) cp_async4(&ring[d + e], src[0] + i0 + e);
+              if (s1) cp_async4(&ring[RG * 32 + d + e], src[1] + i0 + e);
+              if constexpr (NS == 3) if (s2) cp_async4(&ring[2 * RG * 32 + d + e], src[2] + i0 + e);
+            }
+          }
         }
       } else {
-        for (int u = tid; u < nq * NS * 32; u += kTlsClThreads) {
-          const int qq = u / (NS * 32), rem = u - qq * (NS * 32), s = rem >> 5, e = rem & 31;
-          if (!src[s]) continue;
-          const int64_t q = q_fill + qq;
-          const int64_t i = (((q << logC) + crank) << 5) + e;
-          if (i < L.n) cp_async4(&ring[(s * RG + (int)(q & (RG - 1))) * 32 + e], src[s] + i);
+        for (uint32_t u = tid; u < nq * 32; u += kTlsFillThreads) {
+          const uint32_t q = q_fill + (u >> 5), e = u & 31;
+          const uint32_t i = (((q << logC) + (uint32_t)crank) << 5) + e;
+          const int d = (int)(q & (RG - 1)) * 32 + (int)e;
+          if (i < n32) {
+            if (s0) cp_async4(&ring[d], src[0] + i);
+            if (s1) cp_async4(&ring[RG * 32 + d], src[1] + i);
+            if constexpr (NS == 3) if (s2) cp_async4(&ring[2 * RG * 32 + d], src[2] + i);
+          }
         }
       }
       if constexpr (GUIDED) {
-        for (int u = tid; u < nq; u += kTlsClThreads) {
-          const int64_t q = q_fill + u, g = (q << logC) + crank;
+        for (uint32_t u = tid; u < nq; u += kTlsFillThreads) {
+          const uint32_t q = q_fill + u, g = (q << logC) + (uint32_t)crank;
           cp_async4(&bring[q & (RG - 1)], gbits + g);
           cp_async4(&bring[RG + (q & (RG - 1))], gbits + ngroups + g);
         }
       }
-      q_fill = q_to;
     }
+    if (q_to > q_fill) q_fill = q_to;
     cp_async_commit();
   };
 
@@ -632,8 +646,9 @@ __global__ void __launch_bounds__(kTlsClThreads, 1)
   cl_arrive();
   cl_wait();
 
-  int64_t ws = 0;
-  int64_t W = P.window > 0 ? P.window : next_window(L.n, P.prof_raw, -1, P.w_max);
+  uint32_t ws = 0;
+  int W = (int)(P.window > 0 ? P.window : next_window(L.n, P.prof_raw, -1, P.w_max));
+  const int wfix = (int)P.window, wmax = (int)P.w_max;
   long long committed = 0, executed = 0, windows = 0, viol = 0;
   uint32_t epoch = 1;
   int par = 0;
@@ -641,44 +656,44 @@ __global__ void __launch_bounds__(kTlsClThreads, 1)
 #ifdef JP_TLS_TRACE
   const bool trc = crank == 0 && tid == 0;
 #endif
-  while (ws < L.n) {
+  while (ws < n32) {
 #ifdef JP_TLS_TRACE
     const bool tr = trc && windows < kTraceWin;
 #endif
     TLS_TR(0);
-    const int64_t span = W < L.n - ws ? W : L.n - ws;
+    const int span = (int)((uint32_t)W < n32 - ws ? (uint32_t)W : n32 - ws);
     if (tid == 0) s_fv[par] = 0xFFFFFFFFu;   // read last in window-2 (before two cluster barriers)
     refill(ws);
     const unsigned long long tagS = (unsigned long long)(~epoch) << 32;
     const unsigned long long tagC = (unsigned long long)epoch << 32;
     // this CTA's groups in the window: g = q*C + crank, q in [q0, q1)
-    const int64_t g0 = ws >> 5, g1 = (ws + span + 31) >> 5;
-    const int64_t q0 = (g0 + C - 1 - crank) >> logC;   // first q with q*C + crank >= g0
-    const int64_t q1 = (g1 + C - 1 - crank) >> logC;
+    const uint32_t g0 = ws >> 5, g1 = (ws + (uint32_t)span + 31) >> 5;
+    const uint32_t q0 = (g0 + (uint32_t)(C - 1 - crank)) >> logC;   // first q with q*C + crank >= g0
+    const uint32_t q1 = (g1 + (uint32_t)(C - 1 - crank)) >> logC;
     uint32_t va[K], vt[K];
     int32_t wa[K], wt[K], ra[K], rb[K];
     uint32_t offk[K];
     bool act[K], rawk[K];
     // slots of this warp with a group in the window (warp-uniform)
-    const int64_t nq_w = q1 - q0 - warp;
-    const int nk = nq_w <= 0 ? 0 : (int)((nq_w + kTlsClWarps - 1) / kTlsClWarps) < K
-                                     ? (int)((nq_w + kTlsClWarps - 1) / kTlsClWarps) : K;
+    const int nq_w = (int)(q1 - q0) - warp;
+    const int nk = nq_w <= 0 ? 0 : (nq_w + kTlsClWarps - 1) / kTlsClWarps < K ? (nq_w + kTlsClWarps - 1) / kTlsClWarps : K;
     // ---------------- SE: indices, guide bits, stamps ----------------
 #pragma unroll
     for (int k = 0; k < K; k++) {
       if (k >= nk) break;
-      const int64_t q = q0 + warp + (int64_t)k * kTlsClWarps;
+      const uint32_t q = q0 + (uint32_t)(warp + k * kTlsClWarps);
       act[k] = false;
       rawk[k] = false;
       if (q < q1) {                                  // warp-uniform
-        const int64_t i = (((q << logC) + crank) << 5) + lane;
-        act[k] = i >= ws && i < ws + span;
+        const uint32_t i = (((q << logC) + (uint32_t)crank) << 5) + (uint32_t)lane;
+        act[k] = i >= ws && i < ws + (uint32_t)span;
         const int slot = (int)(q & (RG - 1)) * 32 + lane;
-        const int32_t i0 = src[0] ? ring[slot] : (int32_t)(L.ioff + i);
-        const int32_t i1 = src[1] ? ring[RG * 32 + slot] : (int32_t)(L.ioff + i);
+        const int32_t id = (int32_t)L.ioff + (int32_t)i;
+        const int32_t i0 = s0 ? ring[slot] : id;
+        const int32_t i1 = s1 ? ring[RG * 32 + slot] : id;
         int32_t i2 = 0;
-        if constexpr (NS == 3) i2 = src[2] ? ring[2 * RG * 32 + slot] : (int32_t)(L.ioff + i);
-        offk[k] = (uint32_t)(i - ws);
+        if constexpr (NS == 3) i2 = s2 ? ring[2 * RG * 32 + slot] : id;
+        offk[k] = i - ws;
         wa[k] = i1;
         if constexpr (OP == JP_OP_PRIV_TMP) wt[k] = i2;
         if constexpr (OP == JP_OP_SAXPY) ra[k] = i1; else ra[k] = i0;
@@ -719,7 +734,7 @@ __global__ void __launch_bounds__(kTlsClThreads, 1)
     cl_wait();
     TLS_TR(2);
     // ---------------- DC ----------------
-    int64_t fv = span;
+    int fv = span;
     if (dc) {
       unsigned long long sv[K], sv2[K];
 #pragma unroll
@@ -760,7 +775,7 @@ __global__ void __launch_bounds__(kTlsClThreads, 1)
       cl_wait();
       TLS_TR(4);
       const uint32_t f = *(volatile uint32_t *)&s_fv[par];
-      fv = (int64_t)f < span ? (int64_t)f : span;
+      fv = f < (uint32_t)span ? (int)f : span;
     }
     // ---------------- commit [ws, ws+fv) ----------------
     if constexpr (WAW) {
@@ -768,7 +783,7 @@ __global__ void __launch_bounds__(kTlsClThreads, 1)
 #pragma unroll
       for (int k = 0; k < K; k++) {
         if (k >= nk) break;
-        const int64_t q = q0 + warp + (int64_t)k * kTlsClWarps;
+        const uint32_t q = q0 + (uint32_t)(warp + k * kTlsClWarps);
         winA[k] = winT[k] = false;
         if (q < q1) {
           const bool c = act[k] && offk[k] < (uint32_t)fv;
@@ -820,8 +835,8 @@ __global__ void __launch_bounds__(kTlsClThreads, 1)
     TLS_TR(7);
     first = false;
     committed += fv; executed += span; windows++; viol += fv < span;
-    ws += fv;
-    W = P.window > 0 ? P.window : next_window(L.n, P.prof_raw, fv, P.w_max);
+    ws += (uint32_t)fv;
+    W = wfix > 0 ? wfix : next_window_step(fv, wmax);
     epoch++;
     par ^= 1;
   }
