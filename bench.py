@@ -119,10 +119,15 @@ def barrier(world):
     torch.cuda.synchronize()
 
 
+def _coll_dev(dev):
+    # NCCL reduces device tensors; the gloo test mode (JP_DIST_BACKEND=gloo) host ones
+    return dev if torch.distributed.get_backend() == "nccl" else "cpu"
+
+
 def max_over_ranks(x: float, world: int, dev) -> float:
     if world == 1:
         return x
-    t = torch.tensor([x], dtype=torch.float64, device=dev)
+    t = torch.tensor([x], dtype=torch.float64, device=_coll_dev(dev))
     torch.distributed.all_reduce(t, op=torch.distributed.ReduceOp.MAX)
     return float(t.item())
 
@@ -130,7 +135,7 @@ def max_over_ranks(x: float, world: int, dev) -> float:
 def sum_over_ranks(x: float, world: int, dev) -> float:
     if world == 1:
         return x
-    t = torch.tensor([x], dtype=torch.float64, device=dev)
+    t = torch.tensor([x], dtype=torch.float64, device=_coll_dev(dev))
     torch.distributed.all_reduce(t)
     return float(t.item())
 
@@ -304,16 +309,60 @@ def modes_sweep(jp, dev, st):
     return out
 
 
+def partitioned_config4(jp, dev, st, world, rank, steps):
+    """Config 4 (PRIV_TMP fp32, N = 2^26, S = 1024) under task sharing across the
+    ranks.  Profile (local stamp -> C1 MAX over 2 x 4 KiB -> local classify ->
+    C3) timed separately from execution; one step = the
+    privatized execution: local stream -> C4 (MAX over the 8 KiB packed keys)
+    -> finalize.  Barrier, events on the launching stream, max over ranks."""
+    import synth
+    from paper_conf_icpp_hanzlw13_b200 import dist as jd
+    wl = synth.config4(device=dev)
+    full = jp.Loop.from_workload(wl)
+    b, e = jd.sharing_ranges(wl.n, world)[rank]
+    loop = full.range(b, e)
+    ws = jp.workspace(loop)
+
+    def timed(fn, k):
+        for _ in range(3):
+            fn()
+        barrier(world)
+        t0 = torch.cuda.Event(enable_timing=True)
+        t1 = torch.cuda.Event(enable_timing=True)
+        t0.record(st)
+        for _ in range(k):
+            fn()
+        t1.record(st)
+        barrier(world)
+        return max_over_ranks(t0.elapsed_time(t1) / k, world, dev)
+
+    prof = {}
+    prof_ms = timed(lambda: prof.update(jd.profile_partitioned(loop, ws)), steps)
+    mode = jp.jp_select_mode(loop, prof, 0.25)
+    ms = timed(lambda: jd.privatized_partitioned(loop, ws, prof), steps)
+    hbm, _ = peaks()
+    return {"workload": "config4: PRIV_TMP fp32 N=2^26 S=1024, task sharing; step = privatized stream + C4 + finalize",
+            "n": wl.n, "n_per_rank": e - b, "mode": jp.MODE_NAMES[mode], "ms": ms, "iters_per_s": wl.n / (ms * 1e-3),
+            "per_rank_frac_of_hbm": BYTES_PER_ITER_PRIV * (e - b) / (ms * 1e-3) / 1e9 / hbm,
+            "profile_ms": prof_ms, "collective": "torch.distributed all_reduce MAX (C4, 8 KiB int64)"}
+
+
 def run_jp(args):
     import paper_conf_icpp_hanzlw13_b200 as jp
     import synth
     world, rank, local = dist_env()
     if world != args.gpus:
         raise SystemExit(f"--gpus {args.gpus} but WORLD_SIZE={world}: launch N>1 with torchrun")
-    dev = torch.device("cuda", local)
+    # one process per GPU over NCCL; JP_DIST_BACKEND=gloo lets several ranks share
+    # the GPUs of a smaller box to exercise the multi-rank code path (test mode)
+    backend = os.environ.get("JP_DIST_BACKEND", "nccl")
+    dev = torch.device("cuda", local % torch.cuda.device_count())
     torch.cuda.set_device(dev)
     if world > 1:
-        torch.distributed.init_process_group("nccl", device_id=dev)
+        if backend == "nccl":
+            torch.distributed.init_process_group("nccl", device_id=dev)
+        else:
+            torch.distributed.init_process_group(backend)
     st = torch.cuda.current_stream()
     # task sharing: equal weights on identical B200s (P:L354-358, reading A15)
     s0, s1 = jp.jp_plan_sharing(N2, world)[rank]
@@ -381,10 +430,15 @@ def run_jp(args):
                             "algorithmic_bytes_per_iter": BYTES_PER_ITER_SAXPY, "peak_source": peak_src,
                             "kernel_ms": kernel_ms},
                "clocks": clk.summary(), "e2e": e2e, "gpu_launches": launches_all}
-    if world == 1 and not args.no_modes:
+    if not args.no_modes:
         del wl, L
         torch.cuda.empty_cache()
-        out["modes"] = modes_sweep(jp, dev, st)
+        part = partitioned_config4(jp, dev, st, world, rank, 5)
+        torch.cuda.empty_cache()
+        if rank == 0:
+            out["partitioned"] = {"config4": part}
+        if world == 1:
+            out["modes"] = modes_sweep(jp, dev, st)
     if rank == 0:
         out["cpu_baseline"] = oracle_baseline(1 << 25)
         print(json.dumps(out), flush=True)

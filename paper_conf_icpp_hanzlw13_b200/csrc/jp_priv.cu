@@ -230,10 +230,18 @@ __global__ void k_apply_keys(uint32_t *arr, int64_t len, const unsigned long lon
 static bool al16(const void *p) { return ((uintptr_t)p & 15) == 0; }
 
 template <int OP, int DT>
-static void run_priv(const DLoop &d, unsigned long long *kA, unsigned long long *kT, cudaStream_t st, int max_ctas) {
+static void run_priv(const DLoop &d0, unsigned long long *kA, unsigned long long *kT, cudaStream_t st, int max_ctas) {
   int grid = num_sms() * 2;
   if (max_ctas > 0 && grid > max_ctas) grid = max_ctas;
   if constexpr (OP == JP_OP_PRIV_TMP) {
+    // a rank-local range (B1): X and Y are reached only through identity
+    // indices, so rebase them to the range's first element
+    DLoop d = d0;
+    if (!d.r && !d.w && d.ioff > 0) {
+      d.X += d.ioff; d.lenX -= d.ioff;
+      d.A += d.ioff; d.lenA -= d.ioff;
+      d.ioff = 0;
+    }
     if (!d.r && !d.w && d.s && d.ioff == 0 && kT && !kA && d.lenT <= kSmemSlots && al16(d.X) && al16(d.s) &&
         al16(d.A)) {
       if (doall_kernel_choice() == 1) {   // bulk-copy staged (the DOALL kernel choice covers both streams)
@@ -255,6 +263,7 @@ static void run_priv(const DLoop &d, unsigned long long *kA, unsigned long long 
       return;
     }
   }
+  const DLoop &d = d0;
   int smA = kA && d.lenA <= kSmemSlots, smT = kT && d.lenT <= kSmemSlots;
   size_t smem = ((smA ? d.lenA : 0) + (smT ? d.lenT : 0)) * 4;
   int64_t need = (d.n + kPrivThreads - 1) / kPrivThreads;
