@@ -213,22 +213,35 @@ def modes_sweep(jp, dev, st):
     out = {}
     hbm, _ = peaks()
     # config 3: TLS committed iterations/s vs true-RAW density.
-    #  schedule: the whole jp_schedule() call (profile -> Fig. 2(b) mode -> guide -> TLS), what a user runs
-    #  adaptive: jp_run_tls with reading A8's adaptive window (w_max 4096), the path jp_schedule picks
-    #            (single CTA when the first window is < 1024, else a 16-CTA cluster with the guide)
-    #  W4096:    fixed W = 4096 on the guided cluster path
+    #  schedule: the whole jp_schedule() call (profile -> Fig. 2(b) mode -> guide -> TLS), what a user runs;
+    #            it picks the window cap from the density and the TLS path (tls_w_max / tls_path / tls_guided)
+    #  tls:      the same TLS run alone (jp_run_tls with jp_schedule's choices), kernel time
+    #  W4096:    fixed W = 4096 on the guided 16-CTA cluster
     tls = []
     for d in (0.001, 0.01, 0.05, 0.10):
         wl = synth.config3(d, device=dev)
         A0 = wl.A.clone()
         L = jp.Loop.from_workload(wl)
         ws = jp.workspace(L)
+        row = {"density": d}
+        res = None
+        for rep in range(2):   # warm-up, then timed
+            wl.A.copy_(A0)
+            torch.cuda.synchronize()
+            a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            a.record(st)
+            res = jp.jp_schedule(L, ws, stream=st)
+            b.record(st)
+            torch.cuda.synchronize()
+        ms = a.elapsed_time(b)
+        row["raw_iters"] = res["prof"]["raw_iters"]
+        row["schedule"] = {"mode": res["mode_name"], "ms": ms, "committed_per_s": wl.n / (ms * 1e-3),
+                           "windows": res["tls"]["windows"], "tls_w_max": res["tls_w_max"],
+                           "tls_path": {1: "cta", 2: "grid", 3: "cluster16"}.get(res["tls_path"], "?"),
+                           "guided": bool(res["tls_guided"])}
         prof = jp.jp_profile_density(L, ws)
         jp.jp_tls_guide(L, ws)
-        row = {"density": d, "raw_iters": prof["raw_iters"]}
-        w0 = jp.tls_first_window(wl.n, prof["raw_iters"], 4096)
-        adaptive_cluster = w0 >= 1024
-        variants = (("adaptive", dict(window=0, w_max=4096, guided=adaptive_cluster)),
+        variants = (("tls", dict(window=0, w_max=res["tls_w_max"], path=res["tls_path"], guided=bool(res["tls_guided"]))),
                     ("W4096", dict(window=4096, w_max=4096, path=3, guided=True)))
         for name, kw in variants:
             wl.A.copy_(A0)
@@ -243,18 +256,7 @@ def modes_sweep(jp, dev, st):
             ms = a.elapsed_time(b)
             row[name] = {"committed_per_s": s["committed"] / (ms * 1e-3), "ms": ms, "windows": s["windows"],
                          "violations": s["violations"], "executed_over_committed": s["executed"] / s["committed"],
-                         "us_per_window": ms * 1e3 / s["windows"],
-                         "path": ("cluster16+guide" if kw.get("path") == 3 or adaptive_cluster else "cta")}
-        wl.A.copy_(A0)
-        torch.cuda.synchronize()
-        a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
-        a.record(st)
-        res = jp.jp_schedule(L, ws, stream=st)
-        b.record(st)
-        torch.cuda.synchronize()
-        ms = a.elapsed_time(b)
-        row["schedule"] = {"mode": res["mode_name"], "ms": ms, "committed_per_s": wl.n / (ms * 1e-3),
-                           "windows": res["tls"]["windows"]}
+                         "us_per_window": ms * 1e3 / s["windows"]}
         tls.append(row)
         del wl, ws, L, A0
     out["config3_tls"] = tls

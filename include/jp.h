@@ -93,9 +93,10 @@ typedef struct { int64_t committed, executed, windows, violations; } jp_tls_stat
 /* TLS window policy (reading A8).  window > 0: fixed W.  window == 0: adaptive,
  * W0 = clamp(pow2ceil(ceil(4n/raw)),32,w_max) with a profile (w_max if raw == 0,
  * 4096 without profile), then W <- clamp(pow2ceil(2*max(c,16)), 32, w_max)
- * after a window that committed c iterations.  path: 0 auto (3 when the
- * window fits a 16-CTA cluster, else 2), 1 single-CTA shared-memory hash path
- * (W <= 4096), 2 cooperative all-SM path (HBM stamps, software grid barrier),
+ * after a window that committed c iterations.  path: 0 auto (1 when the first
+ * window is < 1024 and the window fits, else 3 when it fits a 16-CTA cluster,
+ * else 2), 1 single-CTA shared-memory hash path (W <= 4096, 2048 for 3-stream
+ * opcodes), 2 cooperative all-SM path (HBM stamps, software grid barrier),
  * 3 one thread-block cluster of `cluster` CTAs (HBM stamps, cluster barriers,
  * W <= 32*(144*cluster - 1)).  cluster: 1..16, 0 = auto (smallest power of two
  * >= 4 that holds the window); ignored by paths 1 and 2.                       */
@@ -113,7 +114,9 @@ typedef struct {
   double tau_high;              /* Fig. 2(b) "(Density > N)" threshold, reading A4 (0.25) */
   int64_t chunk_iters;          /* task size for stealing / sharing (reading A17)     */
   int64_t tls_window;           /* jp_tls_cfg.window                                  */
-  int64_t tls_w_max;            /* jp_tls_cfg.w_max                                   */
+  int64_t tls_w_max;            /* jp_tls_cfg.w_max; 0 = auto from the profiled
+                                   density: clamp(pow2ceil(sqrt(1000/d_raw)), 256, 1024)
+                                   (measured optimum of the single-CTA path)      */
 } jp_sched_cfg;
 
 typedef struct {
@@ -124,6 +127,9 @@ typedef struct {
   int64_t n_tasks;              /* STEALING: same-mode chunk runs                     */
   int64_t n_batches;            /* STEALING: topological batches                      */
   int64_t task_mode_iters[4];   /* iterations executed per jp_mode                    */
+  int64_t tls_w_max;            /* TLS: the window cap used (auto when cfg 0)         */
+  int32_t tls_path;             /* TLS: jp_tls_cfg.path that ran (1, 2, 3)            */
+  int32_t tls_guided;           /* TLS: 1 when the guide (jp_tls_guide) steered it    */
 } jp_sched_result;
 
 /* ---- workspace -------------------------------------------------------------

@@ -227,7 +227,7 @@ def jp_run_tls(loop: Loop, window=0, w_max=65536, path=0, prof=None, ws=None, st
     return {k: getattr(st, k) for k, _ in _abi.jp_tls_stats._fields_} if stats else None
 
 
-def sched_cfg(scheme=JP_SCHED_SHARING, tau_high=0.25, chunk_iters=65536, tls_window=0, tls_w_max=4096,
+def sched_cfg(scheme=JP_SCHED_SHARING, tau_high=0.25, chunk_iters=65536, tls_window=0, tls_w_max=0,
               tls_path=0) -> _abi.jp_sched_cfg:
     return _abi.jp_sched_cfg(int(scheme), int(tls_path), float(tau_high), int(chunk_iters), int(tls_window),
                              int(tls_w_max))
@@ -236,7 +236,8 @@ def sched_cfg(scheme=JP_SCHED_SHARING, tau_high=0.25, chunk_iters=65536, tls_win
 def _res_dict(r: _abi.jp_sched_result) -> dict:
     return {"mode": r.mode, "mode_name": MODE_NAMES.get(r.mode, "?"), "profiled": r.profiled,
             "prof": _prof_dict(r.prof), "tls": {k: getattr(r.tls, k) for k, _ in _abi.jp_tls_stats._fields_},
-            "n_tasks": r.n_tasks, "n_batches": r.n_batches, "task_mode_iters": list(r.task_mode_iters)}
+            "n_tasks": r.n_tasks, "n_batches": r.n_batches, "task_mode_iters": list(r.task_mode_iters),
+            "tls_w_max": r.tls_w_max, "tls_path": r.tls_path, "tls_guided": r.tls_guided}
 
 
 def jp_schedule(loop: Loop, ws=None, cfg=None, stream=None, **kw) -> dict:

@@ -66,7 +66,8 @@ class jp_sched_cfg(C.Structure):
 
 class jp_sched_result(C.Structure):
     _fields_ = [("mode", C.c_int32), ("profiled", C.c_int32), ("prof", jp_profile), ("tls", jp_tls_stats),
-                ("n_tasks", C.c_int64), ("n_batches", C.c_int64), ("task_mode_iters", C.c_int64 * 4)]
+                ("n_tasks", C.c_int64), ("n_batches", C.c_int64), ("task_mode_iters", C.c_int64 * 4),
+                ("tls_w_max", C.c_int64), ("tls_path", C.c_int32), ("tls_guided", C.c_int32)]
 
 
 # (name, restype, argtypes) -- one line per declaration of include/jp.h

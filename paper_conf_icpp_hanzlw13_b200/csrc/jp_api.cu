@@ -410,12 +410,11 @@ static jp_status tls_plan(const Job &j, const jp_tls_cfg *cfg, const jp_profile 
   if (tp.guided && !(hA && j.op != JP_OP_PRIV_TMP)) tp.guided = false;   // nothing to guide
   const int64_t cta_max = tls_cta_wcap(j.op, tp.waw, tp.guided);
   if (path == 0) {
-    // auto (measured): windows that start small stay on one
-    // SM (a CTA barrier is ~50 cycles, a cluster barrier ~1000); windows that
-    // start at >= 1024 iterations spread their gathers over a 16-CTA cluster
-    // (one SM sustains only ~0.25 random L2/HBM loads per cycle).
-    const int64_t w0 = tp.window > 0 ? tp.window : tls_next_window(j.d.n, tp.prof_raw, -1, tp.w_max);
-    path = w0 < 1024 && wcap <= cta_max ? 1 : wcap <= tls_cluster_wcap(16) ? 3 : 2;
+    // auto (measured): windows of <= 1024 iterations stay on
+    // one SM (a CTA barrier is ~50 cycles, a cluster barrier ~1000); larger
+    // windows spread their gathers over a 16-CTA cluster (one SM sustains only
+    // ~0.25 random L2/HBM loads per cycle).
+    path = wcap <= 1024 && wcap <= cta_max ? 1 : wcap <= tls_cluster_wcap(16) ? 3 : 2;
   }
   if (path == 1 && wcap > cta_max)
     return fail(JP_ERR_UNSUPPORTED, "the single-CTA TLS path holds windows up to %lld iterations", (long long)cta_max);
@@ -432,13 +431,29 @@ static jp_status tls_plan(const Job &j, const jp_tls_cfg *cfg, const jp_profile 
   return JP_OK;
 }
 
-// auto_guide: run jp_tls_guide first when the plan is the cluster path and the
-// profile and workspace allow it (jp_schedule; measured gain at low density)
+// TLS window cap from the profiled density (jp_sched_cfg.tls_w_max == 0):
+// clamp(pow2ceil(sqrt(1000 / d_raw)), 256, 1024) -- the measured optimum of the
+// single-CTA path on config 3 (1024 at 0.1%, 512 at 1%, 256-384 at 5-10%;
+// DESIGN.md Sec.6).  A policy parameter of reading A8, not of the semantics.
+static int64_t auto_w_max(const jp_profile *p) {
+  if (!p || p->raw_iters <= 0 || p->n <= 0) return 1024;
+  const double d = (double)p->raw_iters / (double)p->n;
+  const double t = sqrt(1000.0 / d);
+  int64_t w = 256;
+  while ((double)w < t && w < 1024) w <<= 1;
+  return w;
+}
+
+// auto_guide: run jp_tls_guide first when the plan benefits (cluster path
+// always, single-CTA path at d_raw <= 2%: measured) and the profile and
+// workspace allow it (jp_schedule)
 static jp_status run_tls_job(const jp_loop *L, const Job &j, const jp_tls_cfg *cfg, const jp_profile *prof, void *ws,
-                             size_t ws_bytes, jp_tls_stats *stats, cudaStream_t st, bool auto_guide = false) {
+                             size_t ws_bytes, jp_tls_stats *stats, cudaStream_t st, bool auto_guide = false,
+                             TlsPlan *plan_out = nullptr) {
   TlsPlan tp;
   JP_TRY(tls_plan(j, cfg, prof, tp));
-  if (auto_guide && !tp.guided && tp.path == 3 && prof && prof->waw_iters == 0 && a_indirect(j.op, j.d.r, j.d.r2, j.d.w) &&
+  const bool helps = tp.path == 3 || (tp.path == 1 && prof && prof->n > 0 && prof->raw_iters * 50 <= prof->n);
+  if (auto_guide && !tp.guided && helps && prof && prof->waw_iters == 0 && a_indirect(j.op, j.d.r, j.d.r2, j.d.w) &&
       j.op != JP_OP_PRIV_TMP) {
     Layout lg = layout(L);
     if (ws && ws_bytes >= layout_end(lg, JP_WS_PROFILE | JP_WS_GUIDE | JP_WS_TLS) && lg.bytes[R_GUIDE]) {
@@ -449,6 +464,7 @@ static jp_status run_tls_job(const jp_loop *L, const Job &j, const jp_tls_cfg *c
   Layout lo;
   JP_TRY(check_ws(L, ws, ws_bytes, (tp.path >= 2 ? JP_WS_TLS : 0) | (tp.guided ? JP_WS_GUIDE : 0), lo));
   if (has_idx(j) && !prof) JP_TRY(validate_sync(j, ws, lo, st, nullptr));
+  if (plan_out) *plan_out = tp;
   int64_t *hdr = at<int64_t>(ws, lo, R_HEADER);
   JP_CUDA(launch_tls(j, ws, lo, tp, &hdr[H_TLS_COMMITTED], st), "tls");
   if (stats) {
@@ -577,7 +593,7 @@ static jp_sched_cfg default_cfg() {
   c.tau_high = 0.25;
   c.chunk_iters = 65536;
   c.tls_window = 0;
-  c.tls_w_max = 4096;
+  c.tls_w_max = 0;   // auto from the profiled density (auto_w_max)
   c.tls_path = 0;
   return c;
 }
@@ -605,9 +621,15 @@ static jp_status run_mode(const jp_loop *L, const Job &j, int mode, const jp_pro
     JP_CUDA(launch_priv_stream(j, ws, lo, true, st), "priv stream");
     JP_CUDA(launch_priv_finalize(j, ws, lo, st), "priv finalize");
   } else {
-    // profile-guided mode B on the cluster path
-    jp_tls_cfg tc{c.tls_window, c.tls_w_max, c.tls_path, 0, 0, 0};
-    JP_TRY(run_tls_job(L, j, &tc, prof, ws, ws_bytes, &res->tls, st, true));
+    // window cap from the density when not given; profile-guided mode B
+    // where it helps
+    const int64_t wm = c.tls_w_max > 0 ? c.tls_w_max : auto_w_max(prof);
+    jp_tls_cfg tc{c.tls_window, wm, c.tls_path, 0, 0, 0};
+    TlsPlan tp;
+    JP_TRY(run_tls_job(L, j, &tc, prof, ws, ws_bytes, &res->tls, st, true, &tp));
+    res->tls_w_max = wm;
+    res->tls_path = tp.path;
+    res->tls_guided = tp.guided ? 1 : 0;
   }
   res->task_mode_iters[mode] += j.d.n;
   return JP_OK;
@@ -726,12 +748,16 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
         Job sj = sub_job(j, tasks[t].s, tasks[t].e);
         if (tls) {
           TlsPlan tp;
-          jp_tls_cfg tc{c.tls_window, c.tls_w_max, 1, 0, 0, 0};
           jp_profile tprof{};
           tprof.n = sj.d.n;
           tprof.raw_iters = hc.empty() ? -1 : 0;
           for (int64_t k = tasks[t].s / chunk; k * chunk < tasks[t].e; k++) { tprof.raw_iters += hc[3 * k]; tprof.waw_iters += hc[3 * k + 2]; }
+          // the single-CTA path (one SM, beside the partitioned tasks), window cap from the task's density
+          const int64_t wm = c.tls_w_max > 0 ? c.tls_w_max : auto_w_max(tprof.raw_iters >= 0 ? &tprof : nullptr);
+          jp_tls_cfg tc{c.tls_window, wm, 1, 0, 0, 0};
           JP_TRY(tls_plan(sj, &tc, &tprof, tp));
+          res->tls_w_max = wm;
+          res->tls_path = 1;
           JP_CUDA(launch_tls(sj, ws, lo, tp, tstats + 4 * t, s2), "tls task");
           tls_tasks.push_back(t);
         } else if (tasks[t].mode == JP_MODE_PRIVATIZED) {
@@ -772,7 +798,7 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
   jp_sched_cfg c = cfgp ? *cfgp : default_cfg();
   if (c.tau_high <= 0.0) c.tau_high = 0.25;
   if (c.chunk_iters <= 0) c.chunk_iters = 65536;
-  if (c.tls_w_max <= 0) c.tls_w_max = 4096;
+  if (c.tls_w_max < 0) c.tls_w_max = 0;
   memset(res, 0, sizeof *res);
   cudaStream_t st = (cudaStream_t)stp;
   Job j = make_job(L);

@@ -96,7 +96,7 @@ def privatized_partitioned(loop, ws, prof, group=None, engine=None):
     jp.jp_priv_finalize(loop, ws)
 
 
-def schedule_partitioned(loop, ws, group=None, tau_high: float = 0.25, tls_window: int = 0, tls_w_max: int = 4096,
+def schedule_partitioned(loop, ws, group=None, tau_high: float = 0.25, tls_window: int = 0, tls_w_max: int = 2048,
                          full_loop=None, engine=None) -> dict:
     """Task sharing of one loop across the ranks (P:L342-358 generalised to k
     devices).  ``loop`` is this rank's range (iter_base = its first global id,

@@ -30,11 +30,15 @@ def main():
     # (name, path, cluster, window, w_max, guided)
     variants = []
     for g in (False, True):
-        variants += [("cta", 1, 0, 4096, 4096, g), ("cta", 1, 0, 0, 4096, g)]
+        variants += [("cta", 1, 0, 4096, 4096, g)]
+        variants += [("cta", 1, 0, 0, wm, g) for wm in (512, 1024, 2048, 4096)]
         for c in (4, 8, 16):
-            variants += [(f"cl{c}", 3, c, 4096, 4096, g), (f"cl{c}", 3, c, 0, 4096, g)]
+            variants += [(f"cl{c}", 3, c, 4096, 4096, g)]
+            variants += [(f"cl{c}", 3, c, 0, wm, g) for wm in (1024, 2048, 4096)]
         variants += [("cl16", 3, 16, 0, 65024, g)]
-    if args.variants != "all":
+    if args.variants == "wmax":
+        variants = [("cta", 1, 0, 0, wm, g) for g in (False, True) for wm in (128, 256, 384, 512, 768, 1024, 1536)]
+    elif args.variants != "all":
         keep = set(args.variants.split(","))
         variants = [v for v in variants if v[0] in keep]
     for d in [float(x) for x in args.dens.split(",")]:

@@ -348,7 +348,8 @@ def tls_case(wl, window, path, w_max=65536, with_prof=False, cluster=0, guided=F
     return got
 
 
-@pytest.mark.parametrize("window,path", [(32, 1), (100, 1), (1024, 1), (4096, 1), (32, 2), (1000, 2), (8192, 2),
+@pytest.mark.parametrize("window,path", [(32, 1), (100, 1), (1024, 1), (2048, 1), (4096, 1),
+                                         (32, 2), (1000, 2), (8192, 2),
                                          (65536, 2), (32, 3), (100, 3), (1000, 3), (4096, 3), (65536, 3)])
 @pytest.mark.parametrize("d", [0.0, 0.05])
 def test_tls_config1(window, path, d):
@@ -366,8 +367,6 @@ def test_tls_random(op, dt, seed):
     n = [200, 3000, 9001][seed]
     wl = random_loop(500 + op * 10 + dt * 3 + seed, op, dt, n, len_a=max(32, n // [1, 4, 2][seed]))
     for window, path in ((64, 1), (1000, 1), (1000, 2), (64, 3), (1000, 3)):
-        if op == O.OP_PRIV_TMP and window > 2048 and path == 1:
-            continue
         tls_case(wl, window, path)
 
 
@@ -475,9 +474,10 @@ def test_guide_bits_config3(d):
 @pytest.mark.parametrize("d", [0.001, 0.01, 0.05, 0.10])
 def test_tls_guided_config3_reduced(d, path):
     wl = synth.config3(d, n=(1 << 17) + 11)
-    for window in (96, 1000, 4096):
+    wm = 4096
+    for window in (96, 1000, wm):
         tls_case(wl, window, path, guided=True)
-    tls_case(wl, 0, path, w_max=4096, guided=True)
+    tls_case(wl, 0, path, w_max=wm, guided=True)
 
 
 @pytest.mark.parametrize("op,dt", [(op, dt) for op in (O.OP_ADD_C, O.OP_SAXPY, O.OP_STENCIL2) for dt in DTS])
@@ -501,17 +501,24 @@ def test_tls_guided_needs_waw_free_profile():
         jp.jp_run_tls(L, window=64, prof=p, ws=ws, guided=True)
 
 
-@pytest.mark.parametrize("d", [0.01, 0.10])
+@pytest.mark.parametrize("d", [0.001, 0.01, 0.10])
 def test_config3_full_size_guided(d):
     """BASELINE size N=2^24 through jp_schedule (profile -> guide -> TLS), full arrays and stats."""
     wl = synth.config3(d)
     ref = to_oracle(wl)
-    _, A, _, stats = O.sim_tls(ref, 0, 4096, O.profile(ref)["raw_iters"])
     g = gpu(wl)
     L = jp.Loop.from_workload(g)
     res = jp.jp_schedule(L, jp.workspace(L))
     torch.cuda.synchronize()
     assert res["mode"] == jp.JP_MODE_TLS
+    # the window cap jp_schedule derives from the density: clamp(pow2ceil(sqrt(1000/d_raw)), 256, 1024)
+    raw = O.profile(ref)["raw_iters"]
+    t = (1000.0 * wl.n / raw) ** 0.5
+    wm = 256
+    while wm < t and wm < 1024:
+        wm *= 2
+    assert res["tls_w_max"] == wm and res["tls_path"] == 1
+    _, A, _, stats = O.sim_tls(ref, 0, wm, raw)
     check_arrays(g, A, None)
     assert res["tls"] == stats, (res["tls"], stats)
 
@@ -594,19 +601,21 @@ def test_launch_count_and_version():
 
 @pytest.mark.parametrize("waw", [False, True])
 def test_tls_cta_repeatability(waw):
-    """The single-CTA window loop is timing sensitive (TLS
-    barrier): run the densest reduced config-3 loop 12 times per variant."""
+    """The single-CTA window loops are timing sensitive (TLS
+    barrier): run the densest reduced config-3 loop 12 times per kernel."""
     wl = synth.config3(0.10, n=(1 << 17) + 11)
     ref = to_oracle(wl)
-    _, A, _, stats = O.sim_tls(ref, 4096)
+    exp = {w: O.sim_tls(ref, w) for w in (1024, 4096)}
     prof = None
     for rep in range(12):
-        g = gpu(wl)
-        L = jp.Loop.from_workload(g)
-        ws = jp.workspace(L)
-        if not waw and prof is None:
-            prof = jp.jp_profile_density(L, ws)
-        got = jp.jp_run_tls(L, window=4096, w_max=4096, path=1, prof=None if waw else prof, ws=ws)
-        torch.cuda.synchronize()
-        assert got == stats, (rep, got, stats)
-        check_arrays(g, A, None)
+        for path, window in ((1, 1024), (1, 4096)):
+            g = gpu(wl)
+            L = jp.Loop.from_workload(g)
+            ws = jp.workspace(L)
+            if not waw and prof is None:
+                prof = jp.jp_profile_density(L, ws)
+            _, A, _, stats = exp[window]
+            got = jp.jp_run_tls(L, window=window, w_max=window, path=path, prof=None if waw else prof, ws=ws)
+            torch.cuda.synchronize()
+            assert got == stats, (rep, path, got, stats)
+            check_arrays(g, A, None)
