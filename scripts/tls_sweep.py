@@ -36,7 +36,9 @@ def main():
             variants += [(f"cl{c}", 3, c, 4096, 4096, g)]
             variants += [(f"cl{c}", 3, c, 0, wm, g) for wm in (1024, 2048, 4096)]
         variants += [("cl16", 3, 16, 0, 65024, g)]
-    if args.variants == "wmax":
+    if args.variants == "small":
+        variants = [("cta", 1, 0, 0, wm, g) for g in (False, True) for wm in (256, 512, 1024)]
+    elif args.variants == "wmax":
         variants = [("cta", 1, 0, 0, wm, g) for g in (False, True) for wm in (128, 256, 384, 512, 768, 1024, 1536)]
     elif args.variants != "all":
         keep = set(args.variants.split(","))
