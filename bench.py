@@ -291,7 +291,17 @@ def modes_sweep(jp, dev, st):
             jp.jp_schedule(L, ws, stream=st)
             torch.cuda.synchronize()
             ts.append(time.perf_counter() - t0)
-        c1[f"d{d}"] = {"mode": res["mode_name"], "us_per_call": statistics.median(ts) * 1e6}
+        # the CPU oracle on the same loop (sequential run, one host thread) for context
+        import oracle as O
+        ref = O.Loop(wl.op, wl.dtype, wl.n, wl.A.cpu().numpy(), r=wl.r.cpu().numpy(), w=wl.w.cpu().numpy(), c0=wl.c0)
+        to = []
+        for _ in range(20):
+            t0 = time.perf_counter()
+            O.run_seq_inplace(ref)
+            to.append(time.perf_counter() - t0)
+        c1[f"d{d}"] = {"mode": res["mode_name"], "us_per_call": statistics.median(ts) * 1e6,
+                       "path": "tiny (one CTA: profile + mode + run, one launch)" if res.get("profiled") else "",
+                       "oracle_us_per_call": statistics.median(to) * 1e6}
     out["config1"] = c1
     # config 5: mixed, stealing scheme on one GPU (per-chunk profile, tasks, concurrent batch)
     wl = synth.config5(device=dev)

@@ -226,13 +226,30 @@ static jp_status need_device() {
   return JP_OK;
 }
 
+// Small device->host reads of results (a few hundred bytes) go through a
+// per-thread pinned staging buffer: a pageable destination would add a staged
+// copy to every jp_schedule / profile / TLS call (latency-bound config 1).
+static cudaError_t d2h_small_sync(void *dst, const void *src, size_t bytes, cudaStream_t st) {
+  thread_local void *pin = nullptr;
+  thread_local size_t pin_bytes = 0;
+  if (bytes > pin_bytes) {
+    if (pin) cudaFreeHost(pin);
+    pin_bytes = bytes < 4096 ? 4096 : bytes;
+    cudaError_t e = cudaMallocHost(&pin, pin_bytes);
+    if (e != cudaSuccess) { pin = nullptr; pin_bytes = 0; return e; }
+  }
+  cudaError_t e = cudaMemcpyAsync(pin, src, bytes, cudaMemcpyDeviceToHost, st);
+  if (e == cudaSuccess) e = cudaStreamSynchronize(st);
+  if (e == cudaSuccess) memcpy(dst, pin, bytes);
+  return e;
+}
+
 // validate indices on the device, syncs; JP_ERR_INDEX when any is out of range
 static jp_status validate_sync(const Job &j, void *ws, const Layout &lo, cudaStream_t st, int64_t *bad_out) {
   int64_t *hdr = at<int64_t>(ws, lo, R_HEADER);
   JP_CUDA(launch_validate(j, hdr, st), "validate");
   int64_t bad = 0;
-  JP_CUDA(cudaMemcpyAsync(&bad, &hdr[H_BAD], sizeof bad, cudaMemcpyDeviceToHost, st), "validate D2H");
-  JP_CUDA(cudaStreamSynchronize(st), "validate sync");
+  JP_CUDA(d2h_small_sync(&bad, &hdr[H_BAD], sizeof bad, st), "validate D2H");
   if (bad_out) *bad_out = bad;
   if (bad) return fail(JP_ERR_INDEX, "%lld index entries are outside their arrays", (long long)bad);
   return JP_OK;
@@ -305,8 +322,7 @@ jp_status jp_profile_classify(const jp_loop *L, void *ws, size_t ws_bytes, uint3
   cudaStream_t st = (cudaStream_t)stp;
   JP_CUDA(launch_prof_classify(make_job(L), ws, lo, raw_bits, chunk_iters, chunk_counts, st), "profile classify");
   int64_t h[8];
-  JP_CUDA(cudaMemcpyAsync(h, at<int64_t>(ws, lo, R_HEADER), sizeof h, cudaMemcpyDeviceToHost, st), "profile D2H");
-  JP_CUDA(cudaStreamSynchronize(st), "profile sync");
+  JP_CUDA(d2h_small_sync(h, at<int64_t>(ws, lo, R_HEADER), sizeof h, st), "profile D2H");
   if (h[H_BAD]) return fail(JP_ERR_INDEX, "%lld index entries are outside their arrays", (long long)h[H_BAD]);
   fill_profile(out, L->n, h);
   return JP_OK;
@@ -469,8 +485,7 @@ static jp_status run_tls_job(const jp_loop *L, const Job &j, const jp_tls_cfg *c
   JP_CUDA(launch_tls(j, ws, lo, tp, &hdr[H_TLS_COMMITTED], st), "tls");
   if (stats) {
     int64_t h[4];
-    JP_CUDA(cudaMemcpyAsync(h, &hdr[H_TLS_COMMITTED], sizeof h, cudaMemcpyDeviceToHost, st), "tls D2H");
-    JP_CUDA(cudaStreamSynchronize(st), "tls sync");
+    JP_CUDA(d2h_small_sync(h, &hdr[H_TLS_COMMITTED], sizeof h, st), "tls D2H");
     stats->committed = h[0];
     stats->executed = h[1];
     stats->windows = h[2];
@@ -815,6 +830,32 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
   }
   if (c.scheme == JP_SCHED_STEALING) return schedule_stealing(L, j, c, ws, ws_bytes, res, st);
   if (c.scheme != JP_SCHED_SHARING) return fail(JP_ERR_ARG, "bad scheme %d", c.scheme);
+  if (c.tls_path == 0 && c.tls_window <= 4096 && tiny_eligible(L)) {
+    // tiny loop: profile, Fig. 2(b) and the mode in one launch (jp_tiny.cu)
+    Layout lo;
+    JP_TRY(check_ws(L, ws, ws_bytes, 0, lo));
+    int64_t *hdr = at<int64_t>(ws, lo, R_HEADER);
+    JP_CUDA(launch_tiny(j, L, c.tau_high, c.tls_window, c.tls_w_max, hdr, st), "tiny");
+    int64_t h[16];
+    JP_CUDA(d2h_small_sync(h, hdr, sizeof h, st), "tiny D2H");
+    if (h[H_TINY_MODE] < 0) return fail(JP_ERR_INDEX, "%lld index entries are outside their arrays", (long long)h[H_BAD]);
+    fill_profile(&res->prof, L->n, h);
+    res->profiled = 1;
+    res->mode = (int32_t)h[H_TINY_MODE];
+    res->n_tasks = 1;
+    res->n_batches = 1;
+    const int run = res->mode == JP_MODE_SEQ_RECOMMENDED ? JP_MODE_TLS : res->mode;
+    res->task_mode_iters[run] = L->n;
+    if (run == JP_MODE_TLS) {
+      res->tls.committed = h[H_TLS_COMMITTED];
+      res->tls.executed = h[H_TLS_EXECUTED];
+      res->tls.windows = h[H_TLS_WINDOWS];
+      res->tls.violations = h[H_TLS_VIOL];
+      res->tls_w_max = h[H_TINY_WMAX];
+      res->tls_path = 4;
+    }
+    return JP_OK;
+  }
   jp_profile p;
   JP_TRY(jp_profile_density(L, ws, ws_bytes, nullptr, 0, nullptr, &p, stp));
   res->prof = p;

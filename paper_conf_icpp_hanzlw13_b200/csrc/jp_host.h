@@ -65,6 +65,11 @@ cudaError_t launch_task_conflicts(const Job &j, const int32_t *chunk_task, int64
                                   unsigned long long *wmT, unsigned long long *rmT,
                                   unsigned long long *conf, cudaStream_t st);
 
+// tiny loops (jp_tiny.cu): the whole schedule in one CTA's shared memory
+bool tiny_eligible(const jp_loop *L);
+cudaError_t launch_tiny(const Job &j, const jp_loop *L, double tau, int64_t window, int64_t w_max, int64_t *hdr,
+                        cudaStream_t st);
+
 struct TlsPlan {
   int64_t window, w_max, prof_raw;  // prof_raw < 0: no profile
   bool waw;                         // in-window WAW resolution needed

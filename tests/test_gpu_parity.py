@@ -619,3 +619,75 @@ def test_tls_cta_repeatability(waw):
             torch.cuda.synchronize()
             assert got == stats, (rep, path, got, stats)
             check_arrays(g, A, None)
+
+
+# ---------------------------------------------------------------------------
+# tiny loops: the whole schedule in one CTA (jp_tiny.cu)
+# ---------------------------------------------------------------------------
+def tiny_case(wl, expect_mode=None):
+    ref = to_oracle(wl)
+    _, A, T = O.run_seq(ref)
+    p = O.profile(ref)
+    g = gpu(wl)
+    L = jp.Loop.from_workload(g)
+    n0 = jp.jp_launch_count()
+    res = jp.jp_schedule(L, jp.workspace(L))
+    torch.cuda.synchronize()
+    assert jp.jp_launch_count() == n0 + 1           # one launch does profile + mode + run
+    check_arrays(g, A, T)
+    got = (res["prof"]["raw_iters"], res["prof"]["war_iters"], res["prof"]["waw_iters"], res["prof"]["first_raw_iter"])
+    assert got == (p["raw_iters"], p["war_iters"], p["waw_iters"], p["first_raw_iter"])
+    if expect_mode is not None:
+        assert res["mode"] == expect_mode
+    if res["mode"] in (jp.JP_MODE_TLS, jp.JP_MODE_SEQ_RECOMMENDED):
+        assert res["tls_path"] == 4
+        _, A2, _, stats = O.sim_tls(ref, 0, res["tls_w_max"], p["raw_iters"])
+        assert res["tls"] == stats, (res["tls"], stats)
+    return res
+
+
+@pytest.mark.parametrize("d", [0.0, 0.05])
+def test_tiny_config1(d):
+    res = tiny_case(synth.config1(d), jp.JP_MODE_DOALL if d == 0 else jp.JP_MODE_TLS)
+    if d:
+        assert res["prof"]["raw_iters"] == 205
+
+
+@pytest.mark.parametrize("op,dt,seed", [(op, dt, s) for op in OPS for dt in DTS for s in range(4)])
+def test_tiny_random(op, dt, seed):
+    """Random tiny loops of every opcode: every mode appears (duplicate writes ->
+    WAW, small arrays -> RAW/WAR, permutations -> DOALL)."""
+    n = [37, 1000, 4096, 3000][seed]
+    la = [64, 8192, 4096, 3 * 3000][seed] if op != O.OP_PRIV_TMP else max(n, 64)
+    wl = random_loop(4000 + op * 10 + dt * 5 + seed, op, dt, n, len_a=min(la, 8192), null_prob=0.15,
+                     dup_writes=seed != 3, slots=[4, 64, 4096, 1000][seed])
+    tiny_case(wl)
+
+
+def test_tiny_modes_all_reached():
+    """Fig. 2(b) branches inside the tiny kernel: DOALL, PRIVATIZED, TLS, SEQ_RECOMMENDED."""
+    n = 2048
+    ar = torch.arange(n, dtype=torch.int32)
+    perm = torch.from_numpy(np.random.default_rng(3).permutation(n).astype(np.int32))
+    cases = [(synth.Workload("doall", 0, 0, n, ar.clone(), r=perm, w=perm, c0=3), jp.JP_MODE_DOALL),
+             (synth.Workload("war", 0, 0, n, ar.clone(), r=torch.clamp(ar + 1, max=n - 1), w=ar.clone(), c0=3),
+              jp.JP_MODE_PRIVATIZED),
+             (synth.config1(0.05), jp.JP_MODE_TLS),
+             (synth.Workload("chain", 0, 0, n, ar.clone(), r=torch.clamp(ar - 1, min=0), w=ar.clone(), c0=3),
+              jp.JP_MODE_SEQ_RECOMMENDED)]
+    for wl, mode in cases:
+        tiny_case(wl, mode)
+
+
+def test_tiny_bad_index_no_side_effects():
+    wl = synth.config1(0.05)
+    wl.r = wl.r.clone()
+    wl.r[100] = 4096   # out of range
+    g = gpu(wl)
+    A0 = g.A.clone()
+    L = jp.Loop.from_workload(g)
+    with pytest.raises(jp.JPError) as e:
+        jp.jp_schedule(L, jp.workspace(L))
+    assert e.value.status == -5
+    torch.cuda.synchronize()
+    assert torch.equal(g.A, A0)
