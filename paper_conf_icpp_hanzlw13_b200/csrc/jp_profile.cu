@@ -54,8 +54,10 @@ __device__ __forceinline__ int4 idx4(const DLoop &L, const int32_t *p, int64_t i
   return r;
 }
 __device__ __forceinline__ int q4(const int4 &v, int k) { return k == 0 ? v.x : k == 1 ? v.y : k == 2 ? v.z : v.w; }
-__device__ __forceinline__ void stamp32(int32_t *g, int32_t *s, int32_t a, int32_t len, int32_t e, int &bad) {
-  if ((uint32_t)a >= (uint32_t)len) { bad++; return; }
+// chk: the index came from an index array (identity indices were range-checked on the host)
+__device__ __forceinline__ void stamp32(int32_t *g, int32_t *s, int32_t a, int32_t len, int32_t e, int &bad,
+                                        bool chk = true) {
+  if (chk && (uint32_t)a >= (uint32_t)len) { bad++; return; }
   if (s) {
     if (s[a] < e) atomicMax(&s[a], e);
   } else if (g) {
@@ -77,6 +79,8 @@ __global__ void __launch_bounds__(256) k_prof_stamp4(DLoop L, Tabs t, int vec, i
   for (int64_t k = threadIdx.x; k < p - sm; k += blockDim.x) sm[k] = -1;
   JP_CTA_SYNC();
   const int32_t lenA = (int32_t)L.lenA, lenX = (int32_t)L.lenX, lenT = (int32_t)L.lenT;
+  const bool hr = L.r != nullptr, hw = L.w != nullptr,
+             h2 = (OP == JP_OP_STENCIL2 ? L.r2 : OP == JP_OP_PRIV_TMP ? L.s : nullptr) != nullptr;
   int bad = 0;
   const int64_t nq = (L.n + 3) >> 2, B = blockDim.x;
   for (int64_t q0 = (int64_t)blockIdx.x * B * kQuadSteps + threadIdx.x; q0 < nq; q0 += (int64_t)gridDim.x * B * kQuadSteps) {
@@ -102,26 +106,32 @@ __global__ void __launch_bounds__(256) k_prof_stamp4(DLoop L, Tabs t, int vec, i
         if (k >= kn) break;
         const int32_t e = e0 - k;
         const int32_t a = q4(va[u], k), b = q4(vb[u], k);
+        // identity streams (NULL arrays) were range-checked on the host and
+        // reach a table only when the array is also reached through an index
         if constexpr (OP == JP_OP_ADD_C) {
-          stamp32(t.wA, sAw, a, lenA, e, bad);
-          stamp32(t.rA, sAr, b, lenA, e, bad);
+          stamp32(t.wA, sAw, a, lenA, e, bad, hw);
+          stamp32(t.rA, sAr, b, lenA, e, bad, hr);
         } else if constexpr (OP == JP_OP_SAXPY) {
-          if ((uint32_t)b >= (uint32_t)lenX) bad++;
-          stamp32(t.wA, sAw, a, lenA, e, bad);
-          if ((uint32_t)a < (uint32_t)lenA) stamp32(t.rA, sAr, a, lenA, e, bad);
-        } else if constexpr (OP == JP_OP_PRIV_TMP) {
-          if ((uint32_t)b >= (uint32_t)lenX) bad++;
-          if (sTw) {
-            stamp32(t.wT, sTw, a, lenT, e, bad);
-          } else {
-            stamp32(t.wT, nullptr, a, lenT, e, bad);
-            if ((uint32_t)a < (uint32_t)lenT) stamp32(t.rT, nullptr, a, lenT, e, bad);
+          if (hr && (uint32_t)b >= (uint32_t)lenX) bad++;
+          if (hw) {
+            stamp32(t.wA, sAw, a, lenA, e, bad);
+            if ((uint32_t)a < (uint32_t)lenA) stamp32(t.rA, sAr, a, lenA, e, bad, false);
           }
-          stamp32(t.wA, sAw, q4(vc[u], k), lenA, e, bad);
+        } else if constexpr (OP == JP_OP_PRIV_TMP) {
+          if (hr && (uint32_t)b >= (uint32_t)lenX) bad++;
+          if (h2) {
+            if (sTw) {
+              stamp32(t.wT, sTw, a, lenT, e, bad);
+            } else {
+              stamp32(t.wT, nullptr, a, lenT, e, bad);
+              if ((uint32_t)a < (uint32_t)lenT) stamp32(t.rT, nullptr, a, lenT, e, bad, false);
+            }
+          }
+          if (hw) stamp32(t.wA, sAw, q4(vc[u], k), lenA, e, bad);
         } else {
-          stamp32(t.wA, sAw, a, lenA, e, bad);
-          stamp32(t.rA, sAr, b, lenA, e, bad);
-          stamp32(t.rA, sAr, q4(vc[u], k), lenA, e, bad);
+          stamp32(t.wA, sAw, a, lenA, e, bad, hw);
+          stamp32(t.rA, sAr, b, lenA, e, bad, hr);
+          stamp32(t.rA, sAr, q4(vc[u], k), lenA, e, bad, h2);
         }
       }
     }
