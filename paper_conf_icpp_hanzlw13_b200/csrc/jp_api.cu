@@ -392,9 +392,21 @@ jp_status jp_priv_finalize(const jp_loop *L, void *ws, size_t ws_bytes, jp_strea
   return JP_OK;
 }
 
-jp_status jp_run_privatized(const jp_loop *L, const jp_profile *p, void *ws, size_t ws_bytes, jp_stream_t st) {
-  JP_TRY(jp_priv_stream(L, p, ws, ws_bytes, 1, st));
-  return jp_priv_finalize(L, ws, ws_bytes, st);
+jp_status jp_run_privatized(const jp_loop *L, const jp_profile *p, void *ws, size_t ws_bytes, jp_stream_t stp) {
+  JP_TRY(check_loop(L));
+  if (p && p->raw_iters)
+    return fail(JP_ERR_ILLEGAL_MODE, "privatization needs d_raw = 0 (profile: %lld RAW iterations)",
+                (long long)p->raw_iters);
+  JP_TRY(need_device());
+  Layout lo;
+  JP_TRY(check_ws(L, ws, ws_bytes, JP_WS_PRIV, lo));
+  cudaStream_t st = (cudaStream_t)stp;
+  Job j = make_job(L);
+  if (has_idx(j) && !p) JP_TRY(validate_sync(j, ws, lo, st, nullptr));
+  bool applied = false;   // single GPU: the stream kernel may apply the keys itself
+  JP_CUDA(launch_priv_stream(j, ws, lo, true, st, 0, true, &applied), "priv stream");
+  if (!applied) JP_CUDA(launch_priv_finalize(j, ws, lo, st), "priv finalize");
+  return JP_OK;
 }
 
 jp_status jp_tls_guide(const jp_loop *L, void *ws, size_t ws_bytes, jp_stream_t st) {
@@ -633,8 +645,9 @@ static jp_status run_mode(const jp_loop *L, const Job &j, int mode, const jp_pro
     JP_CUDA(launch_doall(j, st), "doall");
   } else if (mode == JP_MODE_PRIVATIZED) {
     if (ws_bytes < layout_end(lo, JP_WS_PRIV)) return fail(JP_ERR_WORKSPACE, "workspace too small for privatization");
-    JP_CUDA(launch_priv_stream(j, ws, lo, true, st), "priv stream");
-    JP_CUDA(launch_priv_finalize(j, ws, lo, st), "priv finalize");
+    bool applied = false;
+    JP_CUDA(launch_priv_stream(j, ws, lo, true, st, 0, true, &applied), "priv stream");
+    if (!applied) JP_CUDA(launch_priv_finalize(j, ws, lo, st), "priv finalize");
   } else {
     // window cap from the density when not given; profile-guided mode B
     // where it helps

@@ -53,8 +53,10 @@ cudaError_t launch_prof_classify(const Job &j, void *ws, const Layout &lo, uint3
 cudaError_t launch_doall(const Job &j, cudaStream_t st, int max_ctas = 0);
 int doall_kernel_choice();
 void set_doall_kernel_choice(int v);
+// fuse_apply: the stream kernel may also apply the keys (single-GPU PE(V));
+// *applied tells whether it did (then launch_priv_finalize is not needed)
 cudaError_t launch_priv_stream(const Job &j, void *ws, const Layout &lo, bool clear_keys,
-                               cudaStream_t st, int max_ctas = 0);
+                               cudaStream_t st, int max_ctas = 0, bool fuse_apply = false, bool *applied = nullptr);
 cudaError_t launch_priv_finalize(const Job &j, void *ws, const Layout &lo, cudaStream_t st);
 cudaError_t launch_merge_apply(void *arr, int64_t len, const int64_t *keys, cudaStream_t st);
 // STEALING scheduler helpers (jp_sched.cu): per-task write/read bitmasks of every

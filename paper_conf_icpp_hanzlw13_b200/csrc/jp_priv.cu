@@ -17,7 +17,10 @@
 // touch fails the plain shared-memory check without issuing an atomic; the
 // flush then recomputes the winner's value and issues one 64-bit global
 // atomicMax per (CTA, touched slot).
+#include <cooperative_groups.h>
 #include "jp_host.h"
+
+namespace cg = cooperative_groups;
 
 namespace jp {
 
@@ -145,8 +148,13 @@ __global__ void __launch_bounds__(kPrivThreads) k_priv_tmp_vec(DLoop L, unsigned
 // too, so the check-before-atomic filter keeps working).
 constexpr int kPrivTile = 4096, kPrivStages = 4, kPrivTmaThreads = 256;
 
+// fuse_apply (cooperative launch, one CTA per SM): after every CTA's flush a
+// grid-wide barrier, then the merged keys are applied to T in the same kernel
+// (R1 + R2 in one launch, single-GPU jp_run_privatized only: across GPUs the
+// keys are merged by C4 between the stream and the finalize).
 template <int DT>
-__global__ void __launch_bounds__(kPrivTmaThreads, 1) k_priv_tmp_tma(DLoop L, unsigned long long *kT, int64_t ntiles) {
+__global__ void __launch_bounds__(kPrivTmaThreads, 1) k_priv_tmp_tma(DLoop L, unsigned long long *kT, int64_t ntiles,
+                                                                     int fuse_apply) {
   extern __shared__ __align__(128) uint32_t psm[];   // [stage][2][tile] then tT[lenT]
   __shared__ __align__(8) unsigned long long full[kPrivStages];
   uint32_t *tT = psm + (size_t)kPrivStages * 2 * kPrivTile;
@@ -217,6 +225,13 @@ __global__ void __launch_bounds__(kPrivTmaThreads, 1) k_priv_tmp_tma(DLoop L, un
     const uint32_t e = tT[b];
     if (e) atomicMax(&kT[b], pack_key(L.base + e - 1, op_mul<DT>(L.c0, L.X[e - 1])));
   }
+  if (fuse_apply) {
+    cg::this_grid().sync();   // every CTA's keys are in
+    for (int64_t b = (int64_t)blockIdx.x * kPrivTmaThreads + tid; b < L.lenT; b += (int64_t)gridDim.x * kPrivTmaThreads) {
+      const unsigned long long k = __ldcg(&kT[b]);
+      if (k) L.T[b] = (uint32_t)k;
+    }
+  }
 }
 
 __global__ void k_apply_keys(uint32_t *arr, int64_t len, const unsigned long long *keys) {
@@ -230,7 +245,8 @@ __global__ void k_apply_keys(uint32_t *arr, int64_t len, const unsigned long lon
 static bool al16(const void *p) { return ((uintptr_t)p & 15) == 0; }
 
 template <int OP, int DT>
-static void run_priv(const DLoop &d0, unsigned long long *kA, unsigned long long *kT, cudaStream_t st, int max_ctas) {
+static void run_priv(const DLoop &d0, unsigned long long *kA, unsigned long long *kT, cudaStream_t st, int max_ctas,
+                     bool fuse_apply, bool *applied) {
   int grid = num_sms() * 2;
   if (max_ctas > 0 && grid > max_ctas) grid = max_ctas;
   if constexpr (OP == JP_OP_PRIV_TMP) {
@@ -251,7 +267,16 @@ static void run_priv(const DLoop &d0, unsigned long long *kA, unsigned long long
         int g = num_sms();
         if (max_ctas > 0 && g > max_ctas) g = max_ctas;
         if (ntiles < g) g = (int)(ntiles < 1 ? 1 : ntiles);
-        k_priv_tmp_tma<DT><<<g, kPrivTmaThreads, smem, st>>>(d, kT, ntiles);
+        int fuse = fuse_apply ? 1 : 0;
+        if (fuse) {   // one CTA per SM: co-resident, as a cooperative launch requires
+          DLoop dd = d;
+          int64_t nt = ntiles;
+          void *args[] = {&dd, &kT, &nt, &fuse};
+          cudaLaunchCooperativeKernel((void *)k_priv_tmp_tma<DT>, dim3(g), dim3(kPrivTmaThreads), args, smem, st);
+          *applied = true;
+        } else {
+          k_priv_tmp_tma<DT><<<g, kPrivTmaThreads, smem, st>>>(d, kT, ntiles, 0);
+        }
         note_launch();
         return;
       }
@@ -273,7 +298,10 @@ static void run_priv(const DLoop &d0, unsigned long long *kA, unsigned long long
 }
 
 cudaError_t launch_priv_stream(const Job &j, void *ws, const Layout &lo, bool clear_keys, cudaStream_t st,
-                               int max_ctas) {
+                               int max_ctas, bool fuse_apply, bool *applied) {
+  bool dummy = false;
+  if (!applied) applied = &dummy;
+  *applied = false;
   auto *kA = at<unsigned long long>(ws, lo, R_KEYS_A);
   auto *kT = at<unsigned long long>(ws, lo, R_KEYS_T);
   if (clear_keys) {
@@ -281,7 +309,7 @@ cudaError_t launch_priv_stream(const Job &j, void *ws, const Layout &lo, bool cl
     if (kT) cudaMemsetAsync(kT, 0, lo.bytes[R_KEYS_T], st);
   }
   if (j.d.n == 0) return launch_check();
-  JP_DISPATCH(j.op, j.dt, run_priv, j.d, kA, kT, st, max_ctas);
+  JP_DISPATCH(j.op, j.dt, run_priv, j.d, kA, kT, st, max_ctas, fuse_apply, applied);
   return launch_check();
 }
 
