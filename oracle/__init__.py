@@ -6,5 +6,5 @@ Only ``tests/``, ``__graft_entry__.smoke()`` and ``bench.py``'s ``cpu_baseline``
 """
 from .oracle import (  # noqa: F401
     OP_ADD_C, OP_SAXPY, OP_PRIV_TMP, OP_STENCIL2, I32, F32, OK, ERR_INDEX,
-    Loop, run_seq, run_seq_inplace, run_order, profile, pairs, raw_sources, sim_tls, tls_next_window, sim_priv, build,
+    Loop, run_seq, run_seq_inplace, run_order, profile, pairs, raw_sources, sim_tls, sim_tls_fwd, tls_next_window, sim_priv, build,
 )

@@ -282,6 +282,41 @@ int jpo_sim_tls(const jpo_loop *L, int64_t window, int64_t w_max, int64_t prof_r
 }
 
 /* ---------------------------------------------------------------------------
+ * TLS with on-chip recovery (reading B7).  P:L320-333 lists the four phases of
+ * a sub-loop: SE, DC, commit of the threads "not found to have violations",
+ * and mis-speculation recovery.  Written as its definition: DC over the window
+ * exactly as in jpo_sim_tls but without stopping at the first violator (every
+ * violating iteration is counted), then the window's iterations take effect
+ * in program order -- the state a correct recovery must reach.
+ * ------------------------------------------------------------------------- */
+int jpo_sim_tls_fwd(const jpo_loop *L, int64_t window, jpo_tls_stats *st) {
+  if (!op_valid(L) || !st || window <= 0) return JPO_ERR_ARG;
+  int e = check_indices(L); if (e) return e;
+  memset(st, 0, sizeof(*st));
+  int64_t len[3] = {L->len_A, L->len_X, L->len_T};
+  int64_t *wmark[3];
+  for (int k = 0; k < 3; k++) wmark[k] = (int64_t *)calloc(len[k] > 0 ? len[k] : 1, sizeof(int64_t));
+  for (int64_t ws = 0; ws < L->n; ws += window) {
+    int64_t we = ws + window < L->n ? ws + window : L->n;
+    int64_t tag = st->windows + 1, v = 0;
+    for (int64_t i = ws; i < we; i++) {
+      accs_t s; accesses(L, i, &s);
+      int viol = 0;
+      for (int k = 0; k < s.nrexp; k++) if (wmark[s.rexp[k].arr][s.rexp[k].a] == tag) viol = 1;
+      v += viol;
+      for (int k = 0; k < s.nwr; k++) wmark[s.wr[k].arr][s.wr[k].a] = tag;
+    }
+    for (int64_t i = ws; i < we; i++) body(L, i, L->A, L->X, L->A, L->T);
+    st->windows++;
+    st->violations += v;
+    st->executed += (we - ws) + v;
+    st->committed += we - ws;
+  }
+  for (int k = 0; k < 3; k++) free(wmark[k]);
+  return JPO_OK;
+}
+
+/* ---------------------------------------------------------------------------
  * Privatized execution PE(V) (Table I private(list)
  * P:L276; readings A9, A10): exposed reads see the pre-loop snapshot, covered
  * reads see the iteration's own private copy, and after all iterations the

@@ -73,6 +73,15 @@ int jpo_sim_tls(const jpo_loop *L, int64_t window, int64_t w_max,
  * prev_commit < 0 => initial window.                                         */
 int64_t jpo_tls_next_window(int64_t n, int64_t prof_raw_iters, int64_t prev_commit,
                             int64_t w_max);
+/* Windowed TLS with on-chip recovery (reading B7):
+ * fixed windows [kW, (k+1)W).  In each window every iteration speculates
+ * against the memory of the window start (SE); DC marks the iterations with an
+ * exposed read written by an EARLIER iteration of the same window ("which
+ * threads fell in violation"); the non-violators commit and the
+ * violators are recovered, so the window ends in the sequential state.
+ * stats: windows; violations = violating iterations (each re-executed once);
+ * executed = n + violations; committed = n.  window > 0.                    */
+int jpo_sim_tls_fwd(const jpo_loop *L, int64_t window, jpo_tls_stats *st);
 /* Privatized semantics (item 5 / readings A9, A10). */
 int jpo_sim_priv(const jpo_loop *L);
 

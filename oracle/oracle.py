@@ -63,6 +63,7 @@ def _load():
             lib.jpo_pairs.argtypes = [P(_Loop), P(_Profile), C.c_void_p]
             lib.jpo_raw_sources.argtypes = [P(_Loop), C.c_void_p]
             lib.jpo_sim_tls.argtypes = [P(_Loop), C.c_int64, C.c_int64, C.c_int64, P(_TlsStats)]
+            lib.jpo_sim_tls_fwd.argtypes = [P(_Loop), C.c_int64, P(_TlsStats)]
             lib.jpo_tls_next_window.argtypes = [C.c_int64] * 4
             lib.jpo_tls_next_window.restype = C.c_int64
             lib.jpo_sim_priv.argtypes = [P(_Loop)]
@@ -156,6 +157,14 @@ def sim_tls(loop: Loop, window: int, w_max: int = 65536, prof_raw_iters: int = -
     L = loop.copy()
     st = _TlsStats()
     s = _load().jpo_sim_tls(C.byref(L._c()), int(window), int(w_max), int(prof_raw_iters), C.byref(st))
+    return s, L.A, L.T, {k: getattr(st, k) for k, _ in _TlsStats._fields_}
+
+
+def sim_tls_fwd(loop: Loop, window: int):
+    """Windowed TLS with on-chip recovery (reading B7). Returns (status, A', T', stats dict)."""
+    L = loop.copy()
+    st = _TlsStats()
+    s = _load().jpo_sim_tls_fwd(C.byref(L._c()), int(window), C.byref(st))
     return s, L.A, L.T, {k: getattr(st, k) for k, _ in _TlsStats._fields_}
 
 

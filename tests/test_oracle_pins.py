@@ -368,3 +368,98 @@ def test_adaptive_tls_equals_sequential():
     for prof in (-1, raw):
         st, A, _, stats = O.sim_tls(L, 0, 256, prof)
         assert A.tolist() == seq.tolist() and stats["committed"] == n
+
+
+# ----------------------------------------------------------------------------
+# TLS with on-chip recovery (reading B7): jpo_sim_tls_fwd
+# ----------------------------------------------------------------------------
+def _sub_loop(L, b, e):
+    """Iterations [b, e) of L as a loop of their own (index arrays sliced)."""
+    sl = lambda a: None if a is None else a[b:e]  # noqa: E731
+    return O.Loop(L.op, L.dtype, e - b, L.A, r=sl(L.r), r2=sl(L.r2), w=sl(L.w), s=sl(L.s), X=L.X, T=L.T,
+                  c0=L.c0, c1=L.c1)
+
+
+def test_tls_fwd_golden(golden_dir):
+    rows = {g["name"]: g for g in load_golden(golden_dir)}
+    with open(os.path.join(golden_dir, "tls_fwd_n8.txt")) as f:
+        for line in f:
+            if line.startswith("#") or not line.strip():
+                continue
+            name, nums = [t.strip() for t in line.split("|")]
+            W, windows, viol, executed, committed = (int(t) for t in nums.split())
+            g = rows[name]
+            L = O.Loop(g["op"], O.I32, 8, g["A0"], r=g["r"], r2=g["r2"], w=g["w"], c0=g["c0"])
+            st, A, _, stats = O.sim_tls_fwd(L, W)
+            assert st == O.OK
+            assert A.tolist() == g["A"].tolist(), name
+            assert (stats["windows"], stats["violations"], stats["executed"], stats["committed"]) == \
+                (windows, viol, executed, committed), name
+
+
+def test_tls_fwd_exhaustive():
+    """N=5, |A|=3, every (r, w), W in {1,2,3,5}: arrays == sequential; the
+    violations of each window are the raw iterations of that window taken as a
+    loop of its own (jpo_profile_run: a different algorithm); W=1 never
+    violates; W >= n gives the whole loop's raw_iters."""
+    n, la = 5, 3
+    A0 = np.array([5, -3, 11], dtype=np.int32)
+    for rw in itertools.product(range(la), repeat=2 * n):
+        L = O.Loop(O.OP_ADD_C, O.I32, n, A0, r=np.array(rw[:n], np.int32), w=np.array(rw[n:], np.int32), c0=7)
+        seq = O.run_seq(L)[1]
+        for W in (1, 2, 3, 5):
+            st, A, _, s = O.sim_tls_fwd(L, W)
+            assert st == O.OK and A.tolist() == seq.tolist()
+            viol = sum(O.profile(_sub_loop(L, b, min(b + W, n)))["raw_iters"] for b in range(0, n, W))
+            assert s == {"committed": n, "executed": n + viol, "windows": -(-n // W), "violations": viol}
+            if W == 1:
+                assert viol == 0
+            if W >= n:
+                assert viol == O.profile(L)["raw_iters"]
+
+
+@pytest.mark.parametrize("op", [O.OP_ADD_C, O.OP_STENCIL2, O.OP_SAXPY, O.OP_PRIV_TMP])
+@pytest.mark.parametrize("dtype", [O.I32, O.F32])
+def test_tls_fwd_random_vs_bruteforce(op, dtype):
+    """Random small loops of every opcode: arrays == sequential, and the
+    violation count equals the pure-Python pair brute force restricted to
+    in-window pairs (j < i in the same window, W(j) ∩ R_exp(i) != {})."""
+    rng = np.random.default_rng(100 + op * 2 + dtype)
+    for trial in range(20):
+        n = int(rng.integers(1, 60))
+        la = int(rng.integers(1, 12))
+        W = int(rng.integers(1, 20))
+        r, r2, w = (rng.integers(0, la, n).astype(np.int32) for _ in range(3))
+        s = rng.integers(0, 4, n).astype(np.int32)
+        el = np.int32 if dtype == O.I32 else np.float32
+        A0 = (rng.integers(-50, 50, la) if dtype == O.I32 else rng.uniform(-1, 1, la)).astype(el)
+        X = (rng.integers(-50, 50, la) if dtype == O.I32 else rng.uniform(-1, 1, la)).astype(el)
+        T0 = np.zeros(4, dtype=el)
+        kw = dict(r=r, w=w)
+        if op == O.OP_STENCIL2:
+            kw["r2"] = r2
+        if op in (O.OP_SAXPY, O.OP_PRIV_TMP):
+            kw["X"] = X
+        if op == O.OP_PRIV_TMP:
+            kw.update(s=s, T=T0)
+        c0 = 3 if dtype == O.I32 else np.float32(1.1)
+        L = O.Loop(op, dtype, n, A0, c0=c0, c1=(2 if dtype == O.I32 else np.float32(0.3)), **kw)
+        _, Aseq, Tseq = O.run_seq(L)
+        st, A, T, stats = O.sim_tls_fwd(L, W)
+        assert st == O.OK
+        assert A.tobytes() == Aseq.tobytes()
+        if op == O.OP_PRIV_TMP:
+            assert T.tobytes() == Tseq.tobytes()
+        sets = [acc_sets(op, i, r, kw.get("r2"), w, kw.get("s")) for i in range(n)]
+        viol = sum(any(set(sets[j][2]) & set(sets[i][0]) for j in range((i // W) * W, i)) for i in range(n))
+        assert stats == {"committed": n, "executed": n + viol, "windows": -(-n // W), "violations": viol}
+
+
+def test_tls_fwd_density_zero_and_args():
+    """d_raw = 0 (a permutation self-update) => no violations at any W; W = 0 is rejected."""
+    n = 300
+    perm = np.random.default_rng(5).permutation(n).astype(np.int32)
+    L = O.Loop(O.OP_ADD_C, O.I32, n, np.arange(n), r=perm, w=perm, c0=1)
+    for W in (1, 7, 64, 1000):
+        assert O.sim_tls_fwd(L, W)[3]["violations"] == 0
+    assert O.sim_tls_fwd(L, 0)[0] == -1
