@@ -100,12 +100,28 @@ typedef struct { int64_t committed, executed, windows, violations; } jp_tls_stat
  * 3 one thread-block cluster of `cluster` CTAs (HBM stamps, cluster barriers,
  * W <= 32*(144*cluster - 1)).  cluster: 1..16, 0 = auto (smallest power of two
  * >= 4 that holds the window); ignored by paths 1 and 2.                       */
+/* Mis-speculation recovery (jp_tls_cfg.recovery).
+ * JP_TLS_RESTART (reading A6): commit the prefix before the first violator and
+ *   restart the next window there; windows per the policy above.
+ * JP_TLS_ONCHIP (reading B7; "commit and mis-speculation recovery",
+ *   P:L373-374): fixed windows [kW, (k+1)W); DC finds EVERY violating iteration
+ *   of the window, the non-violators commit, and each violator is re-executed
+ *   once on chip, in dependence order, with the operand forwarded from its
+ *   writer's shadow slot, so every window commits whole.  Needs a profile with
+ *   waw_iters == 0 (no address written twice; JP_ERR_ARG otherwise).  window:
+ *   fixed W (0 = the largest the cluster holds), W <= 2048*cluster; cluster:
+ *   1..16 (0 = auto: the smallest power of two that holds W, 16 when W = 0 and
+ *   n > 16384); path and w_max are ignored.  stats: windows, violations =
+ *   violating iterations, executed = n + violations, committed = n.  A second
+ *   writer of an address found at run time (a wrong profile) gives JP_ERR_ARG
+ *   after the run, with A in an unspecified state.                          */
+typedef enum { JP_TLS_RESTART = 0, JP_TLS_ONCHIP = 1 } jp_tls_recovery;
 typedef struct {
   int64_t window; int64_t w_max; int32_t path; int32_t cluster;
   int32_t guided;   /* 1: use the guide bitmaps (region 13) that jp_tls_guide wrote for
                        this loop on this workspace; needs a profile with waw_iters == 0
                        (JP_ERR_ARG otherwise).  Same windows, stats and arrays.   */
-  int32_t reserved;
+  int32_t recovery; /* jp_tls_recovery                                          */
 } jp_tls_cfg;
 
 typedef struct {
@@ -117,6 +133,10 @@ typedef struct {
   int64_t tls_w_max;            /* jp_tls_cfg.w_max; 0 = auto from the profiled
                                    density: clamp(pow2ceil(sqrt(1000/d_raw)), 256, 1024)
                                    (measured optimum of the single-CTA path)      */
+  int32_t tls_recovery;         /* 0 auto (JP_TLS_ONCHIP when the profile shows
+                                   waw_iters == 0, else JP_TLS_RESTART), 1 restart,
+                                   2 on-chip                                      */
+  int32_t reserved;
 } jp_sched_cfg;
 
 typedef struct {
@@ -127,9 +147,13 @@ typedef struct {
   int64_t n_tasks;              /* STEALING: same-mode chunk runs                     */
   int64_t n_batches;            /* STEALING: topological batches                      */
   int64_t task_mode_iters[4];   /* iterations executed per jp_mode                    */
-  int64_t tls_w_max;            /* TLS: the window cap used (auto when cfg 0)         */
-  int32_t tls_path;             /* TLS: jp_tls_cfg.path that ran (1, 2, 3)            */
+  int64_t tls_w_max;            /* TLS: the window cap used (auto when cfg 0); the
+                                   fixed window under JP_TLS_ONCHIP                */
+  int32_t tls_path;             /* TLS: jp_tls_cfg.path that ran (1, 2, 3; 4 tiny
+                                   one-CTA schedule; 5 on-chip recovery cluster)  */
   int32_t tls_guided;           /* TLS: 1 when the guide (jp_tls_guide) steered it    */
+  int32_t tls_recovery;         /* TLS: jp_tls_recovery that ran                      */
+  int32_t tls_cluster;          /* TLS: CTAs of the cluster (paths 3 and 5)           */
 } jp_sched_result;
 
 /* ---- workspace -------------------------------------------------------------

@@ -16,7 +16,7 @@ from . import _abi
 from ._abi import (  # noqa: F401
     JP_I32, JP_F32, JP_OP_ADD_C, JP_OP_SAXPY, JP_OP_PRIV_TMP, JP_OP_STENCIL2,
     JP_MODE_DOALL, JP_MODE_PRIVATIZED, JP_MODE_TLS, JP_MODE_SEQ_RECOMMENDED, MODE_NAMES,
-    JP_SCHED_SHARING, JP_SCHED_STEALING, JP_WS_PROFILE, JP_WS_PRIV, JP_WS_TLS, JP_WS_SCHED, JP_WS_GUIDE, JP_WS_ALL,
+    JP_SCHED_SHARING, JP_SCHED_STEALING, JP_TLS_RESTART, JP_TLS_ONCHIP, JP_WS_PROFILE, JP_WS_PRIV, JP_WS_TLS, JP_WS_SCHED, JP_WS_GUIDE, JP_WS_ALL,
     REGIONS, JPError, check, lib,
 )
 
@@ -218,8 +218,9 @@ def jp_tls_guide(loop: Loop, ws: torch.Tensor, stream=None) -> None:
 
 
 def jp_run_tls(loop: Loop, window=0, w_max=65536, path=0, prof=None, ws=None, stats=True, stream=None, cluster=0,
-               guided=False):
-    cfg = _abi.jp_tls_cfg(int(window), int(w_max), int(path), int(cluster), int(bool(guided)), 0)
+               guided=False, recovery=0):
+    """recovery: JP_TLS_RESTART (0, reading A6) or JP_TLS_ONCHIP (1, reading B7)."""
+    cfg = _abi.jp_tls_cfg(int(window), int(w_max), int(path), int(cluster), int(bool(guided)), int(recovery))
     st = _abi.jp_tls_stats()
     p, nb = _ws(ws)
     check(lib().jp_run_tls(loop.ref, C.byref(cfg), _pref(prof), p, nb, C.byref(st) if stats else None,
@@ -228,16 +229,18 @@ def jp_run_tls(loop: Loop, window=0, w_max=65536, path=0, prof=None, ws=None, st
 
 
 def sched_cfg(scheme=JP_SCHED_SHARING, tau_high=0.25, chunk_iters=65536, tls_window=0, tls_w_max=0,
-              tls_path=0) -> _abi.jp_sched_cfg:
+              tls_path=0, tls_recovery=0) -> _abi.jp_sched_cfg:
+    """tls_recovery: 0 auto (on chip when the profile shows waw_iters == 0), 1 restart, 2 on chip."""
     return _abi.jp_sched_cfg(int(scheme), int(tls_path), float(tau_high), int(chunk_iters), int(tls_window),
-                             int(tls_w_max))
+                             int(tls_w_max), int(tls_recovery), 0)
 
 
 def _res_dict(r: _abi.jp_sched_result) -> dict:
     return {"mode": r.mode, "mode_name": MODE_NAMES.get(r.mode, "?"), "profiled": r.profiled,
             "prof": _prof_dict(r.prof), "tls": {k: getattr(r.tls, k) for k, _ in _abi.jp_tls_stats._fields_},
             "n_tasks": r.n_tasks, "n_batches": r.n_batches, "task_mode_iters": list(r.task_mode_iters),
-            "tls_w_max": r.tls_w_max, "tls_path": r.tls_path, "tls_guided": r.tls_guided}
+            "tls_w_max": r.tls_w_max, "tls_path": r.tls_path, "tls_guided": r.tls_guided,
+            "tls_recovery": r.tls_recovery, "tls_cluster": r.tls_cluster}
 
 
 def jp_schedule(loop: Loop, ws=None, cfg=None, stream=None, **kw) -> dict:

@@ -23,6 +23,7 @@ JP_OP_ADD_C, JP_OP_SAXPY, JP_OP_PRIV_TMP, JP_OP_STENCIL2 = 0, 1, 2, 3
 JP_MODE_DOALL, JP_MODE_PRIVATIZED, JP_MODE_TLS, JP_MODE_SEQ_RECOMMENDED = 0, 1, 2, 3
 MODE_NAMES = {0: "DOALL", 1: "PRIVATIZED", 2: "TLS", 3: "SEQ_RECOMMENDED"}
 JP_SCHED_SHARING, JP_SCHED_STEALING = 0, 1
+JP_TLS_RESTART, JP_TLS_ONCHIP = 0, 1
 JP_WS_PROFILE, JP_WS_PRIV, JP_WS_TLS, JP_WS_SCHED, JP_WS_GUIDE, JP_WS_ALL = 1, 2, 4, 8, 16, 31
 REGIONS = {"header": 0, "minW_A": 1, "minR_A": 2, "minW_T": 3, "minR_T": 4, "keys_A": 5, "keys_T": 6,
            "tls_S_A": 7, "tls_C_A": 8, "tls_C_T": 10, "sched": 11, "maxRx_A": 12, "guide": 13}
@@ -56,18 +57,20 @@ class jp_tls_stats(C.Structure):
 
 class jp_tls_cfg(C.Structure):
     _fields_ = [("window", C.c_int64), ("w_max", C.c_int64), ("path", C.c_int32), ("cluster", C.c_int32),
-                ("guided", C.c_int32), ("reserved", C.c_int32)]
+                ("guided", C.c_int32), ("recovery", C.c_int32)]
 
 
 class jp_sched_cfg(C.Structure):
     _fields_ = [("scheme", C.c_int32), ("tls_path", C.c_int32), ("tau_high", C.c_double),
-                ("chunk_iters", C.c_int64), ("tls_window", C.c_int64), ("tls_w_max", C.c_int64)]
+                ("chunk_iters", C.c_int64), ("tls_window", C.c_int64), ("tls_w_max", C.c_int64),
+                ("tls_recovery", C.c_int32), ("reserved", C.c_int32)]
 
 
 class jp_sched_result(C.Structure):
     _fields_ = [("mode", C.c_int32), ("profiled", C.c_int32), ("prof", jp_profile), ("tls", jp_tls_stats),
                 ("n_tasks", C.c_int64), ("n_batches", C.c_int64), ("task_mode_iters", C.c_int64 * 4),
-                ("tls_w_max", C.c_int64), ("tls_path", C.c_int32), ("tls_guided", C.c_int32)]
+                ("tls_w_max", C.c_int64), ("tls_path", C.c_int32), ("tls_guided", C.c_int32),
+                ("tls_recovery", C.c_int32), ("tls_cluster", C.c_int32)]
 
 
 # (name, restype, argtypes) -- one line per declaration of include/jp.h

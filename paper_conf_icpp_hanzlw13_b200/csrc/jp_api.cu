@@ -436,6 +436,35 @@ static jp_status tls_plan(const Job &j, const jp_tls_cfg *cfg, const jp_profile 
   if (tp.guided && (!prof || prof->waw_iters != 0))
     return fail(JP_ERR_ARG, "a guided TLS run needs a profile with waw_iters == 0");
   if (tp.guided && !(hA && j.op != JP_OP_PRIV_TMP)) tp.guided = false;   // nothing to guide
+  tp.recovery = cfg ? cfg->recovery : JP_TLS_RESTART;
+  if (tp.recovery != JP_TLS_RESTART && tp.recovery != JP_TLS_ONCHIP)
+    return fail(JP_ERR_ARG, "bad TLS recovery %d", tp.recovery);
+  if (tp.recovery == JP_TLS_ONCHIP) {
+    // reading B7: one shadow slot per address needs a loop that writes no address twice
+    if (!prof || prof->waw_iters != 0)
+      return fail(JP_ERR_ARG, "on-chip TLS recovery needs a profile with waw_iters == 0");
+    const int cmax = tls_fwd_max_cluster();
+    if (cl > cmax) return fail(JP_ERR_UNSUPPORTED, "the device schedules TLS clusters of up to %d CTAs", cmax);
+    if (tp.window > 0) {
+      if (cl == 0) {
+        cl = 1;
+        while (cl < cmax && tls_fwd_wcap(cl) < tp.window) cl <<= 1;
+      }
+      if (tls_fwd_wcap(cl) < tp.window)
+        return fail(JP_ERR_UNSUPPORTED, "a %d-CTA on-chip TLS cluster holds windows up to %lld iterations", cl,
+                    (long long)tls_fwd_wcap(cl));
+    } else {
+      if (cl == 0) {
+        cl = 1;
+        while (cl < cmax && tls_fwd_wcap(cl) < j.d.n) cl <<= 1;
+      }
+      tp.window = tls_fwd_wcap(cl);
+    }
+    tp.cluster = cl;
+    tp.path = 5;
+    tp.waw = false;
+    return JP_OK;
+  }
   const int64_t cta_max = tls_cta_wcap(j.op, tp.waw, tp.guided);
   if (path == 0) {
     // auto (measured): windows of <= 1024 iterations stay on
@@ -480,7 +509,7 @@ static jp_status run_tls_job(const jp_loop *L, const Job &j, const jp_tls_cfg *c
                              TlsPlan *plan_out = nullptr) {
   TlsPlan tp;
   JP_TRY(tls_plan(j, cfg, prof, tp));
-  const bool helps = tp.path == 3 || (tp.path == 1 && prof && prof->n > 0 && prof->raw_iters * 50 <= prof->n);
+  const bool helps = tp.path == 3 || tp.path == 5 || (tp.path == 1 && prof && prof->n > 0 && prof->raw_iters * 50 <= prof->n);
   if (auto_guide && !tp.guided && helps && prof && prof->waw_iters == 0 && a_indirect(j.op, j.d.r, j.d.r2, j.d.w) &&
       j.op != JP_OP_PRIV_TMP) {
     Layout lg = layout(L);
@@ -490,14 +519,22 @@ static jp_status run_tls_job(const jp_loop *L, const Job &j, const jp_tls_cfg *c
     }
   }
   Layout lo;
-  JP_TRY(check_ws(L, ws, ws_bytes, (tp.path >= 2 ? JP_WS_TLS : 0) | (tp.guided ? JP_WS_GUIDE : 0), lo));
+  const int uses = (tp.path == 2 || tp.path == 3 ? JP_WS_TLS : 0) | (tp.guided ? JP_WS_GUIDE : 0);
+  JP_TRY(check_ws(L, ws, ws_bytes, uses, lo));
   if (has_idx(j) && !prof) JP_TRY(validate_sync(j, ws, lo, st, nullptr));
   if (plan_out) *plan_out = tp;
   int64_t *hdr = at<int64_t>(ws, lo, R_HEADER);
-  JP_CUDA(launch_tls(j, ws, lo, tp, &hdr[H_TLS_COMMITTED], st), "tls");
+  if (tp.path == 5) {
+    const uint32_t *bits = tp.guided ? at<uint32_t>(ws, lo, R_GUIDE) : nullptr;
+    JP_CUDA(launch_tls_fwd(j, tp.window, tp.cluster, bits, &hdr[H_TLS_COMMITTED], st), "tls on-chip");
+  } else {
+    JP_CUDA(launch_tls(j, ws, lo, tp, &hdr[H_TLS_COMMITTED], st), "tls");
+  }
   if (stats) {
     int64_t h[4];
     JP_CUDA(d2h_small_sync(h, &hdr[H_TLS_COMMITTED], sizeof h, st), "tls D2H");
+    if (tp.path == 5 && h[0] < 0)
+      return fail(JP_ERR_ARG, "on-chip TLS recovery met an address written twice (the profile passed was wrong)");
     stats->committed = h[0];
     stats->executed = h[1];
     stats->windows = h[2];
@@ -651,13 +688,19 @@ static jp_status run_mode(const jp_loop *L, const Job &j, int mode, const jp_pro
   } else {
     // window cap from the density when not given; profile-guided mode B
     // where it helps
+    // recovery: on chip (reading B7) whenever the profile allows it, unless asked otherwise
+    const int rec = c.tls_recovery == 1 ? JP_TLS_RESTART
+                    : c.tls_recovery == 2 || (c.tls_path == 0 && prof && prof->waw_iters == 0) ? JP_TLS_ONCHIP
+                                                                                            : JP_TLS_RESTART;
     const int64_t wm = c.tls_w_max > 0 ? c.tls_w_max : auto_w_max(prof);
-    jp_tls_cfg tc{c.tls_window, wm, c.tls_path, 0, 0, 0};
+    jp_tls_cfg tc{c.tls_window, wm, c.tls_path, 0, 0, rec};
     TlsPlan tp;
     JP_TRY(run_tls_job(L, j, &tc, prof, ws, ws_bytes, &res->tls, st, true, &tp));
-    res->tls_w_max = wm;
+    res->tls_w_max = rec == JP_TLS_ONCHIP ? tp.window : wm;
     res->tls_path = tp.path;
     res->tls_guided = tp.guided ? 1 : 0;
+    res->tls_recovery = rec;
+    res->tls_cluster = tp.path == 3 || tp.path == 5 ? tp.cluster : 1;
   }
   res->task_mode_iters[mode] += j.d.n;
   return JP_OK;
@@ -843,7 +886,7 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
   }
   if (c.scheme == JP_SCHED_STEALING) return schedule_stealing(L, j, c, ws, ws_bytes, res, st);
   if (c.scheme != JP_SCHED_SHARING) return fail(JP_ERR_ARG, "bad scheme %d", c.scheme);
-  if (c.tls_path == 0 && c.tls_window <= 4096 && tiny_eligible(L)) {
+  if (c.tls_path == 0 && c.tls_recovery != 2 && c.tls_window <= 4096 && tiny_eligible(L)) {
     // tiny loop: profile, Fig. 2(b) and the mode in one launch (jp_tiny.cu)
     Layout lo;
     JP_TRY(check_ws(L, ws, ws_bytes, 0, lo));

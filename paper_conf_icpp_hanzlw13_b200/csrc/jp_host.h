@@ -75,10 +75,16 @@ cudaError_t launch_tiny(const Job &j, const jp_loop *L, double tau, int64_t wind
 struct TlsPlan {
   int64_t window, w_max, prof_raw;  // prof_raw < 0: no profile
   bool waw;                         // in-window WAW resolution needed
-  int path;                         // 1 cta, 2 grid, 3 cluster
-  int cluster;                      // CTAs of the cluster path (power of two)
+  int path;                         // 1 cta, 2 grid, 3 cluster, 5 on-chip recovery cluster
+  int cluster;                      // CTAs of the cluster paths (power of two)
   bool guided;                      // stamp only RAW sources, check only RAW readers
+  int recovery;                     // jp_tls_recovery
 };
+// on-chip recovery path (jp_tls_fwd.cu, reading B7): fixed window (> 0), cluster of C CTAs
+cudaError_t launch_tls_fwd(const Job &j, int64_t window, int cluster, const uint32_t *bits, int64_t *stats,
+                           cudaStream_t st);
+int64_t tls_fwd_wcap(int cluster);   // largest window a C-CTA cluster holds (2048*C)
+int tls_fwd_max_cluster();           // 16 when the device schedules it, else 8
 // stats: int64[4] device (committed, executed, windows, violations); bar: u32[2]
 // zeroed barrier words + int64[3] fv slots (grid path).
 cudaError_t launch_tls(const Job &j, void *ws, const Layout &lo, const TlsPlan &p, int64_t *stats,

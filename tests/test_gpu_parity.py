@@ -503,12 +503,13 @@ def test_tls_guided_needs_waw_free_profile():
 
 @pytest.mark.parametrize("d", [0.001, 0.01, 0.10])
 def test_config3_full_size_guided(d):
-    """BASELINE size N=2^24 through jp_schedule (profile -> guide -> TLS), full arrays and stats."""
+    """BASELINE size N=2^24 through jp_schedule (profile -> guide -> TLS with restart
+    recovery, tls_recovery = 1), full arrays and stats."""
     wl = synth.config3(d)
     ref = to_oracle(wl)
     g = gpu(wl)
     L = jp.Loop.from_workload(g)
-    res = jp.jp_schedule(L, jp.workspace(L))
+    res = jp.jp_schedule(L, jp.workspace(L), tls_recovery=1)
     torch.cuda.synchronize()
     assert res["mode"] == jp.JP_MODE_TLS
     # the window cap jp_schedule derives from the density: clamp(pow2ceil(sqrt(1000/d_raw)), 256, 1024)

@@ -1,0 +1,189 @@
+"""GPU parity of TLS with on-chip recovery (JP_TLS_ONCHIP, reading B7)
+against oracle/jpo.c jpo_sim_tls_fwd: every output array byte-equal and the
+statistics (windows, violations, executed, committed) exact, through the C ABI.
+
+Loops must write no address twice (profile waw_iters == 0), so the cases are
+the dependent-set generator of configs 1/3 (w a permutation), write-once
+random loops of every opcode, and the full-length dependence chains
+(prefix chain, Gauss-Seidel) that make every iteration of a window wait on
+its predecessor's forwarded value.
+"""
+import numpy as np
+import pytest
+import torch
+
+import oracle as O
+import synth
+from helpers import random_loop, to_oracle
+
+pytestmark = pytest.mark.gpu
+
+if torch.cuda.is_available():
+    import paper_conf_icpp_hanzlw13_b200 as jp
+    DEV = torch.device("cuda:0")
+else:  # collected on CPU boxes, never run there
+    jp = None
+    DEV = None
+
+OPS = [O.OP_ADD_C, O.OP_SAXPY, O.OP_PRIV_TMP, O.OP_STENCIL2]
+DTS = [O.I32, O.F32]
+
+
+def same(t: torch.Tensor, a: np.ndarray) -> bool:
+    return t.cpu().numpy().tobytes() == a.tobytes()
+
+
+def fwd_case(wl, window, cluster=0, guided=False, view=None):
+    """Profile -> (guide) -> on-chip TLS; compare with the oracle.  window = 0:
+    the path's own window (2048 * cluster), returned by the check."""
+    ref = to_oracle(wl)
+    g = wl.to(DEV)
+    L = jp.Loop.from_workload(g) if view is None else view(g)
+    ws = jp.workspace(L)
+    p = jp.jp_profile_density(L, ws)
+    assert p["waw_iters"] == 0
+    if guided:
+        jp.jp_tls_guide(L, ws)
+    got = jp.jp_run_tls(L, window=window, prof=p, ws=ws, cluster=cluster, guided=guided,
+                        recovery=jp.JP_TLS_ONCHIP)
+    torch.cuda.synchronize()
+    W = window
+    if W == 0:
+        c = cluster
+        if c == 0:
+            c = 1
+            while c < 16 and 2048 * c < wl.n:
+                c *= 2
+        W = 2048 * c
+    st, A, T, stats = O.sim_tls_fwd(ref, W)
+    assert st == O.OK
+    assert same(g.A, A), f"A differs at {np.flatnonzero(g.A.cpu().numpy() != A)[:10]}"
+    if T is not None:
+        assert same(g.T, T)
+    assert got == stats, (got, stats)
+    return got
+
+
+@pytest.mark.parametrize("window", [1, 32, 100, 1000, 2048, 4096, 0])
+@pytest.mark.parametrize("d", [0.0, 0.05])
+def test_fwd_config1(window, d):
+    fwd_case(synth.config1(d), window)
+
+
+@pytest.mark.parametrize("cluster", [1, 2, 4, 8, 16])
+def test_fwd_cluster_sizes(cluster):
+    wl = synth.config3(0.05, n=(1 << 15) + 77)
+    for window in (96, 1000, 2048 * cluster):
+        fwd_case(wl, window, cluster=cluster)
+        fwd_case(wl, window, cluster=cluster, guided=True)
+
+
+@pytest.mark.parametrize("d", [0.001, 0.01, 0.05, 0.10])
+@pytest.mark.parametrize("guided", [False, True])
+def test_fwd_config3_reduced(d, guided):
+    wl = synth.config3(d, n=(1 << 17) + 11)
+    for window in (4096, 32768, 0):
+        fwd_case(wl, window, guided=guided)
+
+
+@pytest.mark.parametrize("op,dt", [(op, dt) for op in OPS for dt in DTS])
+def test_fwd_random_write_once(op, dt):
+    """Write-once random loops (w a partial permutation; PRIV_TMP's s too) of every
+    opcode and dtype, NULL indices included, several windows and clusters."""
+    n = 7001
+    wl = random_loop(1300 + op * 10 + dt, op, dt, n, len_a=3 * n, null_prob=0.2, dup_writes=False,
+                     slots=2 * n)
+    for window, cluster in ((64, 0), (1500, 0), (2048, 1), (4096, 2), (0, 0)):
+        fwd_case(wl, window, cluster=cluster)
+        if op != O.OP_PRIV_TMP:
+            fwd_case(wl, window, cluster=cluster, guided=True)
+
+
+def test_fwd_chains():
+    """Every iteration depends on the previous one (prefix chain, Gauss-Seidel):
+    each window resolves a dependence chain as long as the window."""
+    n = 40000
+    A0 = torch.arange(n, dtype=torch.int32) * 3
+    ar = torch.arange(n, dtype=torch.int32)
+    pc = synth.Workload("pc", O.OP_ADD_C, O.I32, n, A0.clone(), r=torch.clamp(ar - 1, min=0), w=ar.clone(), c0=7)
+    for window in (100, 2048, 32768):
+        st = fwd_case(pc, window)
+        assert st["violations"] == n - -(-n // window)
+    gs = synth.Workload("gs", O.OP_STENCIL2, O.F32, n, (A0.float() * 0.01).clone(), r=torch.clamp(ar - 1, min=0),
+                        r2=torch.clamp(ar + 1, max=n - 1), w=ar.clone(), c0=0.4)
+    for window in (777, 32768):
+        fwd_case(gs, window)
+        fwd_case(gs, window, guided=True)
+
+
+def test_fwd_unaligned_views():
+    """Index streams that start 3 entries into their tensors."""
+    n = 9000
+    wl = synth.config3(0.05, n=n + 3)
+    sl = lambda t: None if t is None else t[3:]  # noqa: E731
+    sub = synth.Workload("sub", wl.op, wl.dtype, n, wl.A.clone(), r=sl(wl.r), w=sl(wl.w), c0=wl.c0)
+    view = lambda g: jp.Loop(wl.op, wl.dtype, n, g.A, r=sl(g.r), w=sl(g.w), c0=wl.c0)  # noqa: E731
+    ref = to_oracle(sub)
+    g = wl.to(DEV)
+    L = view(g)
+    ws = jp.workspace(L)
+    p = jp.jp_profile_density(L, ws)
+    got = jp.jp_run_tls(L, window=1000, prof=p, ws=ws, recovery=jp.JP_TLS_ONCHIP)
+    torch.cuda.synchronize()
+    _, A, _, stats = O.sim_tls_fwd(ref, 1000)
+    assert same(g.A, A) and got == stats
+
+
+def test_fwd_repeatability():
+    """Races in the write log or the shadow-slot polls would show as run-to-run differences."""
+    wl = synth.config3(0.10, n=1 << 20)
+    ref = to_oracle(wl)
+    _, A, _, stats = O.sim_tls_fwd(ref, 32768)
+    g = wl.to(DEV)
+    A0 = g.A.clone()
+    L = jp.Loop.from_workload(g)
+    ws = jp.workspace(L)
+    p = jp.jp_profile_density(L, ws)
+    jp.jp_tls_guide(L, ws)
+    for rep in range(10):
+        g.A.copy_(A0)
+        got = jp.jp_run_tls(L, window=32768, prof=p, ws=ws, guided=bool(rep & 1), recovery=jp.JP_TLS_ONCHIP)
+        torch.cuda.synchronize()
+        assert same(g.A, A) and got == stats, rep
+
+
+def test_fwd_needs_write_once_profile():
+    wl = random_loop(5, O.OP_ADD_C, O.I32, 3000, len_a=64, null_prob=0.0)
+    g = wl.to(DEV)
+    L = jp.Loop.from_workload(g)
+    ws = jp.workspace(L)
+    with pytest.raises(jp.JPError):          # no profile
+        jp.jp_run_tls(L, window=64, ws=ws, recovery=jp.JP_TLS_ONCHIP)
+    p = jp.jp_profile_density(L, ws)
+    assert p["waw_iters"] > 0
+    with pytest.raises(jp.JPError):          # profile with WAW
+        jp.jp_run_tls(L, window=64, prof=p, ws=ws, recovery=jp.JP_TLS_ONCHIP)
+    wl3 = synth.config3(0.01, n=1 << 16).to(DEV)
+    L3 = jp.Loop.from_workload(wl3)
+    p3 = jp.jp_profile_density(L3, jp.workspace(L3))
+    with pytest.raises(jp.JPError):          # window larger than a 16-CTA cluster holds
+        jp.jp_run_tls(L3, window=2048 * 16 + 1, prof=p3, ws=jp.workspace(L3), recovery=jp.JP_TLS_ONCHIP)
+    with pytest.raises(jp.JPError):          # window larger than the given cluster holds
+        jp.jp_run_tls(L3, window=4097, cluster=2, prof=p3, ws=jp.workspace(L3), recovery=jp.JP_TLS_ONCHIP)
+
+
+@pytest.mark.parametrize("d", [0.001, 0.01, 0.05, 0.10])
+def test_fwd_config3_full_size_schedule(d):
+    """BASELINE size N=2^24 through jp_schedule (profile -> Fig. 2(b) TLS -> guide ->
+    on-chip recovery, the default for write-once loops): full arrays and stats."""
+    wl = synth.config3(d)
+    ref = to_oracle(wl)
+    g = wl.to(DEV)
+    L = jp.Loop.from_workload(g)
+    res = jp.jp_schedule(L, jp.workspace(L))
+    torch.cuda.synchronize()
+    assert res["mode"] == jp.JP_MODE_TLS and res["tls_recovery"] == jp.JP_TLS_ONCHIP and res["tls_path"] == 5
+    assert res["tls_cluster"] == 16 and res["tls_w_max"] == 32768
+    _, A, _, stats = O.sim_tls_fwd(ref, res["tls_w_max"])
+    assert same(g.A, A)
+    assert res["tls"] == stats, (res["tls"], stats)
