@@ -213,50 +213,55 @@ def modes_sweep(jp, dev, st):
     out = {}
     hbm, _ = peaks()
     # config 3: TLS committed iterations/s vs true-RAW density.
-    #  schedule: the whole jp_schedule() call (profile -> Fig. 2(b) mode -> guide -> TLS), what a user runs;
-    #            it picks the window cap from the density and the TLS path (tls_w_max / tls_path / tls_guided)
-    #  tls:      the same TLS run alone (jp_run_tls with jp_schedule's choices), kernel time
-    #  W4096:    fixed W = 4096 on the guided 16-CTA cluster
+    #  schedule:  the whole jp_schedule() call (profile -> Fig. 2(b) mode -> guide -> TLS), what a user runs;
+    #             on this write-once loop it takes on-chip recovery (reading B7) on every SM
+    #  tls:       that TLS run alone (jp_run_tls with jp_schedule's choices), kernel time
+    #  profile / guide: jp_profile_density and jp_tls_guide alone
+    #  restart_*: the same with restart recovery (reading A6: prefix commit, restart at the first violator)
     tls = []
+    names = {1: "cta", 2: "grid", 3: "cluster16", 4: "tiny", 5: "onchip-cluster", 6: "onchip-grid"}
+
+    def timed(fn, A, A0):
+        out = None
+        for rep in range(2):   # warm-up, then timed
+            A.copy_(A0)
+            torch.cuda.synchronize()
+            a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            a.record(st)
+            out = fn()
+            b.record(st)
+            torch.cuda.synchronize()
+        return out, a.elapsed_time(b)
+
     for d in (0.001, 0.01, 0.05, 0.10):
         wl = synth.config3(d, device=dev)
         A0 = wl.A.clone()
         L = jp.Loop.from_workload(wl)
         ws = jp.workspace(L)
         row = {"density": d}
-        res = None
-        for rep in range(2):   # warm-up, then timed
-            wl.A.copy_(A0)
-            torch.cuda.synchronize()
-            a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
-            a.record(st)
-            res = jp.jp_schedule(L, ws, stream=st)
-            b.record(st)
-            torch.cuda.synchronize()
-        ms = a.elapsed_time(b)
-        row["raw_iters"] = res["prof"]["raw_iters"]
-        row["schedule"] = {"mode": res["mode_name"], "ms": ms, "committed_per_s": wl.n / (ms * 1e-3),
-                           "windows": res["tls"]["windows"], "tls_w_max": res["tls_w_max"],
-                           "tls_path": {1: "cta", 2: "grid", 3: "cluster16"}.get(res["tls_path"], "?"),
-                           "guided": bool(res["tls_guided"])}
-        prof = jp.jp_profile_density(L, ws)
-        jp.jp_tls_guide(L, ws)
-        variants = (("tls", dict(window=0, w_max=res["tls_w_max"], path=res["tls_path"], guided=bool(res["tls_guided"]))),
-                    ("W4096", dict(window=4096, w_max=4096, path=3, guided=True)))
-        for name, kw in variants:
-            wl.A.copy_(A0)
-            jp.jp_run_tls(L, prof=prof, ws=ws, stream=st, **kw)   # warm-up
-            wl.A.copy_(A0)
-            torch.cuda.synchronize()
-            a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
-            a.record(st)
-            s = jp.jp_run_tls(L, prof=prof, ws=ws, stream=st, **kw)
-            b.record(st)
-            torch.cuda.synchronize()
-            ms = a.elapsed_time(b)
-            row[name] = {"committed_per_s": s["committed"] / (ms * 1e-3), "ms": ms, "windows": s["windows"],
-                         "violations": s["violations"], "executed_over_committed": s["executed"] / s["committed"],
-                         "us_per_window": ms * 1e3 / s["windows"]}
+        for tag, rec in (("", 0), ("restart_", 1)):
+            res, ms = timed(lambda: jp.jp_schedule(L, ws, stream=st, tls_recovery=rec), wl.A, A0)
+            row["raw_iters"] = res["prof"]["raw_iters"]
+            row[tag + "schedule"] = {"mode": res["mode_name"], "ms": ms, "committed_per_s": wl.n / (ms * 1e-3),
+                                     "windows": res["tls"]["windows"], "violations": res["tls"]["violations"],
+                                     "recovery": ["restart", "onchip"][res["tls_recovery"]],
+                                     "window" if res["tls_recovery"] else "tls_w_max": res["tls_w_max"],
+                                     "tls_path": names.get(res["tls_path"], "?"), "ctas": res["tls_cluster"],
+                                     "guided": bool(res["tls_guided"])}
+            prof = jp.jp_profile_density(L, ws)
+            if res["tls_guided"]:
+                jp.jp_tls_guide(L, ws)
+            kw = dict(window=res["tls_w_max"], path=res["tls_path"], guided=bool(res["tls_guided"]), recovery=1) \
+                if res["tls_recovery"] else \
+                dict(window=0, w_max=res["tls_w_max"], path=res["tls_path"], guided=bool(res["tls_guided"]))
+            s, ms = timed(lambda: jp.jp_run_tls(L, prof=prof, ws=ws, stream=st, **kw), wl.A, A0)
+            row[tag + "tls"] = {"committed_per_s": s["committed"] / (ms * 1e-3), "ms": ms, "windows": s["windows"],
+                                "violations": s["violations"], "executed_over_committed": s["executed"] / s["committed"],
+                                "us_per_window": ms * 1e3 / s["windows"]}
+        _, ms = timed(lambda: jp.jp_profile_density(L, ws, stream=st), wl.A, A0)
+        row["profile_ms"] = ms
+        _, ms = timed(lambda: jp.jp_tls_guide(L, ws, stream=st), wl.A, A0)
+        row["guide_ms"] = ms
         tls.append(row)
         del wl, ws, L, A0
     out["config3_tls"] = tls

@@ -109,9 +109,12 @@ typedef struct { int64_t committed, executed, windows, violations; } jp_tls_stat
  *   once on chip, in dependence order, with the operand forwarded from its
  *   writer's shadow slot, so every window commits whole.  Needs a profile with
  *   waw_iters == 0 (no address written twice; JP_ERR_ARG otherwise).  window:
- *   fixed W (0 = the largest the cluster holds), W <= 2048*cluster; cluster:
- *   1..16 (0 = auto: the smallest power of two that holds W, 16 when W = 0 and
- *   n > 16384); path and w_max are ignored.  stats: windows, violations =
+ *   fixed W (0 = the largest the path holds); path: 5 one thread-block
+ *   cluster, W <= 2048*cluster, cluster 1..16 (0 = auto: the smallest power of
+ *   two that holds W, or n when W = 0); 6 every SM (cooperative), W <= 2048 *
+ *   co-resident CTAs (303104 on a 148-SM B200), write log and shadow values in
+ *   workspace regions 7 and 8 (JP_WS_TLS); 0 = auto (5 when W, or n if W = 0,
+ *   fits a 16-CTA cluster, else 6).  w_max is ignored.  stats: windows, violations =
  *   violating iterations, executed = n + violations, committed = n.  A second
  *   writer of an address found at run time (a wrong profile) gives JP_ERR_ARG
  *   after the run, with A in an unspecified state.                          */
@@ -150,10 +153,11 @@ typedef struct {
   int64_t tls_w_max;            /* TLS: the window cap used (auto when cfg 0); the
                                    fixed window under JP_TLS_ONCHIP                */
   int32_t tls_path;             /* TLS: jp_tls_cfg.path that ran (1, 2, 3; 4 tiny
-                                   one-CTA schedule; 5 on-chip recovery cluster)  */
+                                   one-CTA schedule; 5 / 6 on-chip recovery on a
+                                   cluster / on every SM)                         */
   int32_t tls_guided;           /* TLS: 1 when the guide (jp_tls_guide) steered it    */
   int32_t tls_recovery;         /* TLS: jp_tls_recovery that ran                      */
-  int32_t tls_cluster;          /* TLS: CTAs of the cluster (paths 3 and 5)           */
+  int32_t tls_cluster;          /* TLS: CTAs of the cluster (paths 3, 5) or grid (6)  */
 } jp_sched_result;
 
 /* ---- workspace -------------------------------------------------------------
@@ -168,7 +172,8 @@ enum { JP_WS_PROFILE = 1, JP_WS_PRIV = 2, JP_WS_TLS = 4, JP_WS_SCHED = 8, JP_WS_
 size_t jp_workspace_bytes(const jp_loop *L /* host */, int32_t uses);
 /* region ids: 0 header, 1 minW(A) int32, 2 minR(A) int32, 3 minW(T), 4 minR(T),
  * 5 keys(A) int64, 6 keys(T) int64, 7 tls stamps(A) u64, 8 tls commit(A) u64,
- * 9 (reserved), 10 tls commit(T) u64, 11 scheduler scratch, 12 latest exposed
+ * 9 (reserved), 10 tls commit(T) u64 (regions 7 and 8 are the write log S[a] and
+ * shadow values V[a] of on-chip TLS recovery on path 6), 11 scheduler scratch, 12 latest exposed
  * reader maxRx(A) int32 (gid, empty -1), 13 TLS guide bitmaps u32 [2][ceil(n/32)]
  * (raw words, then RAW-source words; see jp_tls_guide).  Stamp tables hold
  * INT32_MAX - gid (empty = -1) so that an all_reduce MAX over int32 yields the

@@ -445,6 +445,19 @@ static jp_status tls_plan(const Job &j, const jp_tls_cfg *cfg, const jp_profile 
       return fail(JP_ERR_ARG, "on-chip TLS recovery needs a profile with waw_iters == 0");
     const int cmax = tls_fwd_max_cluster();
     if (cl > cmax) return fail(JP_ERR_UNSUPPORTED, "the device schedules TLS clusters of up to %d CTAs", cmax);
+    if (path != 0 && path != 5 && path != 6) return fail(JP_ERR_ARG, "on-chip TLS runs on path 5 (cluster) or 6 (grid)");
+    // auto: a window the 16-CTA cluster holds stays there, larger loops use every SM
+    if (path == 0) path = (tp.window > 0 ? tp.window : j.d.n) <= tls_fwd_wcap(cmax) ? 5 : 6;
+    if (path == 6) {
+      const int64_t gcap = tls_fwd_grid_wcap();
+      if (tp.window == 0) tp.window = gcap;
+      if (tp.window > gcap)
+        return fail(JP_ERR_UNSUPPORTED, "the on-chip TLS grid holds windows up to %lld iterations", (long long)gcap);
+      tp.cluster = (int)((tp.window + tls_fwd_wcap(1) - 1) / tls_fwd_wcap(1));
+      tp.path = 6;
+      tp.waw = false;
+      return JP_OK;
+    }
     if (tp.window > 0) {
       if (cl == 0) {
         cl = 1;
@@ -506,34 +519,42 @@ static int64_t auto_w_max(const jp_profile *p) {
 // workspace allow it (jp_schedule)
 static jp_status run_tls_job(const jp_loop *L, const Job &j, const jp_tls_cfg *cfg, const jp_profile *prof, void *ws,
                              size_t ws_bytes, jp_tls_stats *stats, cudaStream_t st, bool auto_guide = false,
-                             TlsPlan *plan_out = nullptr) {
+                             TlsPlan *plan_out = nullptr, bool guide_ready = false) {
   TlsPlan tp;
   JP_TRY(tls_plan(j, cfg, prof, tp));
-  const bool helps = tp.path == 3 || tp.path == 5 || (tp.path == 1 && prof && prof->n > 0 && prof->raw_iters * 50 <= prof->n);
+  const bool helps = tp.path == 3 || tp.path >= 5 || (tp.path == 1 && prof && prof->n > 0 && prof->raw_iters * 50 <= prof->n);
   if (auto_guide && !tp.guided && helps && prof && prof->waw_iters == 0 && a_indirect(j.op, j.d.r, j.d.r2, j.d.w) &&
       j.op != JP_OP_PRIV_TMP) {
     Layout lg = layout(L);
     if (ws && ws_bytes >= layout_end(lg, JP_WS_PROFILE | JP_WS_GUIDE | JP_WS_TLS) && lg.bytes[R_GUIDE]) {
-      JP_CUDA(launch_tls_guide(j, ws, lg, st), "tls guide");
+      if (!guide_ready) JP_CUDA(launch_tls_guide(j, ws, lg, st), "tls guide");
       tp.guided = true;
     }
   }
   Layout lo;
-  const int uses = (tp.path == 2 || tp.path == 3 ? JP_WS_TLS : 0) | (tp.guided ? JP_WS_GUIDE : 0);
+  const int uses = (tp.path == 2 || tp.path == 3 || tp.path == 6 ? JP_WS_TLS : 0) | (tp.guided ? JP_WS_GUIDE : 0);
   JP_TRY(check_ws(L, ws, ws_bytes, uses, lo));
   if (has_idx(j) && !prof) JP_TRY(validate_sync(j, ws, lo, st, nullptr));
   if (plan_out) *plan_out = tp;
   int64_t *hdr = at<int64_t>(ws, lo, R_HEADER);
+  const uint32_t *bits = tp.guided ? at<uint32_t>(ws, lo, R_GUIDE) : nullptr;
+  const uint32_t *bsrc = bits ? bits + (L->n + 31) / 32 : nullptr;
   if (tp.path == 5) {
-    const uint32_t *bits = tp.guided ? at<uint32_t>(ws, lo, R_GUIDE) : nullptr;
-    JP_CUDA(launch_tls_fwd(j, tp.window, tp.cluster, bits, &hdr[H_TLS_COMMITTED], st), "tls on-chip");
+    JP_CUDA(launch_tls_fwd(j, tp.window, tp.cluster, bits, bsrc, &hdr[H_TLS_COMMITTED], st), "tls on-chip");
+  } else if (tp.path == 6) {
+    auto *S = at<unsigned long long>(ws, lo, R_TLS_S_A);
+    auto *V = at<unsigned long long>(ws, lo, R_TLS_C_A);
+    const int64_t lenS = S && V ? L->len_A : 0;
+    JP_CUDA(launch_tls_fwd_grid(j, tp.window, bits, bsrc, S, V, lenS, reinterpret_cast<unsigned *>(&hdr[H_BAR_COUNT]),
+                                &hdr[H_TLS_COMMITTED], st),
+            "tls on-chip grid");
   } else {
     JP_CUDA(launch_tls(j, ws, lo, tp, &hdr[H_TLS_COMMITTED], st), "tls");
   }
   if (stats) {
     int64_t h[4];
     JP_CUDA(d2h_small_sync(h, &hdr[H_TLS_COMMITTED], sizeof h, st), "tls D2H");
-    if (tp.path == 5 && h[0] < 0)
+    if (tp.path >= 5 && h[0] < 0)
       return fail(JP_ERR_ARG, "on-chip TLS recovery met an address written twice (the profile passed was wrong)");
     stats->committed = h[0];
     stats->executed = h[1];
@@ -676,7 +697,7 @@ static Job sub_job(const Job &j, int64_t s, int64_t e) {
 }
 
 static jp_status run_mode(const jp_loop *L, const Job &j, int mode, const jp_profile *prof, const jp_sched_cfg &c,
-                          void *ws, size_t ws_bytes, jp_sched_result *res, cudaStream_t st) {
+                          void *ws, size_t ws_bytes, jp_sched_result *res, cudaStream_t st, bool guide_ready = false) {
   Layout lo = layout(L);
   if (mode == JP_MODE_DOALL) {
     JP_CUDA(launch_doall(j, st), "doall");
@@ -695,12 +716,12 @@ static jp_status run_mode(const jp_loop *L, const Job &j, int mode, const jp_pro
     const int64_t wm = c.tls_w_max > 0 ? c.tls_w_max : auto_w_max(prof);
     jp_tls_cfg tc{c.tls_window, wm, c.tls_path, 0, 0, rec};
     TlsPlan tp;
-    JP_TRY(run_tls_job(L, j, &tc, prof, ws, ws_bytes, &res->tls, st, true, &tp));
+    JP_TRY(run_tls_job(L, j, &tc, prof, ws, ws_bytes, &res->tls, st, true, &tp, guide_ready));
     res->tls_w_max = rec == JP_TLS_ONCHIP ? tp.window : wm;
     res->tls_path = tp.path;
     res->tls_guided = tp.guided ? 1 : 0;
     res->tls_recovery = rec;
-    res->tls_cluster = tp.path == 3 || tp.path == 5 ? tp.cluster : 1;
+    res->tls_cluster = tp.path == 3 || tp.path >= 5 ? tp.cluster : 1;
   }
   res->task_mode_iters[mode] += j.d.n;
   return JP_OK;
@@ -794,6 +815,12 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
   // 4. run batch by batch; tasks of one batch are pairwise conflict-free and run
   //    concurrently (TLS on one SM, partitioned modes on the rest)
   int64_t *tstats = reinterpret_cast<int64_t *>(sch + sl.tstats);
+  // guide bitmaps for on-chip TLS tasks (from this profile's stamp tables)
+  bool guided_ok = false;
+  for (int t = 0; t < nt && !guided_ok; t++) guided_ok = tasks[t].mode == JP_MODE_TLS;
+  guided_ok = guided_ok && c.tls_recovery != 1 && lo.bytes[R_GUIDE] && j.op != JP_OP_PRIV_TMP &&
+              a_indirect(j.op, j.d.r, j.d.r2, j.d.w);
+  if (guided_ok) JP_CUDA(launch_tls_guide(j, ws, lo, st), "tls guide");
   cudaEvent_t ev0;
   JP_CUDA(cudaEventCreateWithFlags(&ev0, cudaEventDisableTiming), "event");
   std::vector<cudaEvent_t> evs;
@@ -823,13 +850,31 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
           tprof.n = sj.d.n;
           tprof.raw_iters = hc.empty() ? -1 : 0;
           for (int64_t k = tasks[t].s / chunk; k * chunk < tasks[t].e; k++) { tprof.raw_iters += hc[3 * k]; tprof.waw_iters += hc[3 * k + 2]; }
-          // the single-CTA path (one SM, beside the partitioned tasks), window cap from the task's density
-          const int64_t wm = c.tls_w_max > 0 ? c.tls_w_max : auto_w_max(tprof.raw_iters >= 0 ? &tprof : nullptr);
-          jp_tls_cfg tc{c.tls_window, wm, 1, 0, 0, 0};
-          JP_TRY(tls_plan(sj, &tc, &tprof, tp));
-          res->tls_w_max = wm;
-          res->tls_path = 1;
-          JP_CUDA(launch_tls(sj, ws, lo, tp, tstats + 4 * t, s2), "tls task");
+          const bool onchip = c.tls_recovery == 2 || (c.tls_recovery == 0 && c.tls_path == 0 && tprof.waw_iters == 0);
+          if (onchip) {
+            // on-chip recovery (reading B7) on one cluster beside the partitioned tasks, guided by
+            // the whole loop's bitmaps (the task starts on a chunk boundary, a multiple of 32)
+            jp_tls_cfg tc{c.tls_window, 0, 5, 0, 0, JP_TLS_ONCHIP};
+            JP_TRY(tls_plan(sj, &tc, &tprof, tp));
+            const uint32_t *gb = guided_ok ? at<uint32_t>(ws, lo, R_GUIDE) : nullptr;
+            const int64_t nw = (L->n + 31) / 32;
+            res->tls_w_max = tp.window;
+            res->tls_path = 5;
+            res->tls_recovery = JP_TLS_ONCHIP;
+            res->tls_cluster = tp.cluster;
+            res->tls_guided = gb ? 1 : 0;
+            JP_CUDA(launch_tls_fwd(sj, tp.window, tp.cluster, gb ? gb + tasks[t].s / 32 : nullptr,
+                                   gb ? gb + nw + tasks[t].s / 32 : nullptr, tstats + 4 * t, s2),
+                    "tls task");
+          } else {
+            // the single-CTA path (one SM, beside the partitioned tasks), window cap from the task's density
+            const int64_t wm = c.tls_w_max > 0 ? c.tls_w_max : auto_w_max(tprof.raw_iters >= 0 ? &tprof : nullptr);
+            jp_tls_cfg tc{c.tls_window, wm, 1, 0, 0, 0};
+            JP_TRY(tls_plan(sj, &tc, &tprof, tp));
+            res->tls_w_max = wm;
+            res->tls_path = 1;
+            JP_CUDA(launch_tls(sj, ws, lo, tp, tstats + 4 * t, s2), "tls task");
+          }
           tls_tasks.push_back(t);
         } else if (tasks[t].mode == JP_MODE_PRIVATIZED) {
           JP_CUDA(launch_priv_stream(sj, ws, lo, false, s2), "priv task");
@@ -913,14 +958,27 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
     return JP_OK;
   }
   jp_profile p;
-  JP_TRY(jp_profile_density(L, ws, ws_bytes, nullptr, 0, nullptr, &p, stp));
+  // the classify pass also writes the TLS guide bitmaps when the loop can be guided
+  // (A read through an index, workspace with the guide region): no separate guide pass
+  const Layout lg = layout(L);
+  const bool gfuse = lg.bytes[R_GUIDE] && ws && ws_bytes >= layout_end(lg, JP_WS_PROFILE | JP_WS_GUIDE | JP_WS_TLS);
+  if (gfuse) {
+    JP_TRY(jp_profile_stamp(L, ws, ws_bytes, stp));
+    JP_CUDA(launch_prof_classify_guide(j, ws, lg, st), "profile classify");
+    int64_t h[8];
+    JP_CUDA(d2h_small_sync(h, at<int64_t>(ws, lg, R_HEADER), sizeof h, st), "profile D2H");
+    if (h[H_BAD]) return fail(JP_ERR_INDEX, "%lld index entries are outside their arrays", (long long)h[H_BAD]);
+    fill_profile(&p, L->n, h);
+  } else {
+    JP_TRY(jp_profile_density(L, ws, ws_bytes, nullptr, 0, nullptr, &p, stp));
+  }
   res->prof = p;
   res->profiled = 1;
   res->mode = select_mode_counts(p.n, p.raw_iters, p.war_iters, p.waw_iters, c.tau_high);
   res->n_tasks = 1;
   res->n_batches = 1;
   const int run = res->mode == JP_MODE_SEQ_RECOMMENDED ? JP_MODE_TLS : res->mode;
-  return run_mode(L, j, run, &p, c, ws, ws_bytes, res, st);
+  return run_mode(L, j, run, &p, c, ws, ws_bytes, res, st, gfuse && p.waw_iters == 0);
 }
 
 // ---------------------------------------------------------------------------

@@ -50,6 +50,8 @@ cudaError_t launch_tls_guide(const Job &j, void *ws, const Layout &lo, cudaStrea
 cudaError_t launch_prof_stamp(const Job &j, void *ws, const Layout &lo, cudaStream_t st);
 cudaError_t launch_prof_classify(const Job &j, void *ws, const Layout &lo, uint32_t *raw_bits,
                                  int64_t chunk, int64_t *chunk_counts, cudaStream_t st);
+// counts + the TLS guide bitmaps (region 13, valid when the loop writes no address twice) in one pass
+cudaError_t launch_prof_classify_guide(const Job &j, void *ws, const Layout &lo, cudaStream_t st);
 cudaError_t launch_doall(const Job &j, cudaStream_t st, int max_ctas = 0);
 int doall_kernel_choice();
 void set_doall_kernel_choice(int v);
@@ -81,10 +83,17 @@ struct TlsPlan {
   int recovery;                     // jp_tls_recovery
 };
 // on-chip recovery path (jp_tls_fwd.cu, reading B7): fixed window (> 0), cluster of C CTAs
-cudaError_t launch_tls_fwd(const Job &j, int64_t window, int cluster, const uint32_t *bits, int64_t *stats,
-                           cudaStream_t st);
+// bits / bsrc: guide words (raw readers / RAW sources) of local iteration 0's word, or NULL (unguided)
+cudaError_t launch_tls_fwd(const Job &j, int64_t window, int cluster, const uint32_t *bits, const uint32_t *bsrc,
+                           int64_t *stats, cudaStream_t st);
 int64_t tls_fwd_wcap(int cluster);   // largest window a C-CTA cluster holds (2048*C)
 int tls_fwd_max_cluster();           // 16 when the device schedules it, else 8
+// on-chip recovery over every SM (cooperative): S, V = u64 [lenS] (regions 7, 8), bar = 2 zeroed u32
+cudaError_t launch_tls_fwd_grid(const Job &j, int64_t window, const uint32_t *bits, const uint32_t *bsrc,
+                                unsigned long long *S,
+                                unsigned long long *V, int64_t lenS, unsigned *bar, int64_t *stats,
+                                cudaStream_t st);
+int64_t tls_fwd_grid_wcap();         // 2048 * co-resident CTAs (2048 * 148 on B200)
 // stats: int64[4] device (committed, executed, windows, violations); bar: u32[2]
 // zeroed barrier words + int64[3] fv slots (grid path).
 cudaError_t launch_tls(const Job &j, void *ws, const Layout &lo, const TlsPlan &p, int64_t *stats,

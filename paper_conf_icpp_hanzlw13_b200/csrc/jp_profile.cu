@@ -152,9 +152,16 @@ __global__ void __launch_bounds__(256) k_prof_stamp4(DLoop L, Tabs t, int vec, i
 }
 
 // counts-only classify (no raw bitmap, no chunk counts): per-thread counters,
-// one reduction per CTA
-template <int OP>
-__global__ void __launch_bounds__(256) k_prof_count4(DLoop L, Tabs t, int vec, int64_t *hdr) {
+// one reduction per CTA.  GUIDE: also the TLS guide bitmaps of jp_tls_guide
+// (region 13) in the same pass -- raw words by an OR over the 8 lanes that
+// share a word, and RAW-source words by an atomicOr at each raw read's first
+// writer.  The source words equal jp_tls_guide's whenever the loop writes no
+// address twice (then an address read by a later iteration has exactly one
+// writer, the first), which is the only case a guided TLS run accepts; the
+// caller zeroes them first.
+template <int OP, bool GUIDE>
+__global__ void __launch_bounds__(256) k_prof_count4(DLoop L, Tabs t, int vec, int64_t *hdr, uint32_t *graw,
+                                                     uint32_t *gsrc) {
   __shared__ unsigned long long s_cnt[3];
   __shared__ unsigned long long s_first;
   if (threadIdx.x < 3) s_cnt[threadIdx.x] = 0;
@@ -165,7 +172,14 @@ __global__ void __launch_bounds__(256) k_prof_count4(DLoop L, Tabs t, int vec, i
   unsigned c_raw = 0, c_war = 0, c_waw = 0;
   unsigned long long first = ~0ull;
   const int64_t nq = (L.n + 3) >> 2, B = blockDim.x;
-  for (int64_t q0 = (int64_t)blockIdx.x * B * kQuadSteps + threadIdx.x; q0 < nq; q0 += (int64_t)gridDim.x * B * kQuadSteps) {
+  // the writer (local iteration) behind a raw read of address a: mark it a RAW source
+  auto mark_src = [&](int32_t a) {
+    if constexpr (GUIDE) {
+      const int64_t j = (int64_t)(0x7FFFFFFF - t.wA[a]) - L.base;
+      atomicOr(&gsrc[j >> 5], 1u << (j & 31));
+    }
+  };
+  for (int64_t q0 = (int64_t)blockIdx.x * B * kQuadSteps + threadIdx.x; q0 - threadIdx.x < nq; q0 += (int64_t)gridDim.x * B * kQuadSteps) {
     int4 va[kQuadSteps], vb[kQuadSteps], vc[kQuadSteps];
 #pragma unroll
     for (int u = 0; u < kQuadSteps; u++) {
@@ -181,33 +195,49 @@ __global__ void __launch_bounds__(256) k_prof_count4(DLoop L, Tabs t, int vec, i
 #pragma unroll
     for (int u = 0; u < kQuadSteps; u++) {
       const int64_t q = q0 + u * B;
-      if (q >= nq) break;
-      const int32_t e0 = enc_gid(L.base + (q << 2));
-      const int kn = L.n - (q << 2) < 4 ? (int)(L.n - (q << 2)) : 4;
+      uint32_t rb = 0;   // raw bits of this lane's 4 iterations
+      if (q < nq) {
+        const int32_t e0 = enc_gid(L.base + (q << 2));
+        const int kn = L.n - (q << 2) < 4 ? (int)(L.n - (q << 2)) : 4;
 #pragma unroll
-      for (int k = 0; k < 4; k++) {
-        if (k >= kn) break;
-        const int32_t e = e0 - k;
-        const int32_t a = q4(va[u], k);
-        bool raw = false, war, waw;
-        if constexpr (OP == JP_OP_ADD_C) {
-          raw = earlier32(t.wA, q4(vb[u], k), lenA, e);
-          war = earlier32(t.rA, a, lenA, e);
-          waw = earlier32(t.wA, a, lenA, e);
-        } else if constexpr (OP == JP_OP_SAXPY) {
-          raw = earlier32(t.wA, a, lenA, e);
-          war = earlier32(t.rA, a, lenA, e);
-          waw = raw;
-        } else if constexpr (OP == JP_OP_PRIV_TMP) {
-          war = earlier32(rT, a, lenT, e);
-          waw = earlier32(t.wT, a, lenT, e) || earlier32(t.wA, q4(vb[u], k), lenA, e);
-        } else {
-          raw = earlier32(t.wA, q4(vb[u], k), lenA, e) || earlier32(t.wA, q4(vc[u], k), lenA, e);
-          war = earlier32(t.rA, a, lenA, e);
-          waw = earlier32(t.wA, a, lenA, e);
+        for (int k = 0; k < 4; k++) {
+          if (k >= kn) break;
+          const int32_t e = e0 - k;
+          const int32_t a = q4(va[u], k);
+          bool raw = false, war, waw;
+          if constexpr (OP == JP_OP_ADD_C) {
+            raw = earlier32(t.wA, q4(vb[u], k), lenA, e);
+            war = earlier32(t.rA, a, lenA, e);
+            waw = earlier32(t.wA, a, lenA, e);
+            if (raw) mark_src(q4(vb[u], k));
+          } else if constexpr (OP == JP_OP_SAXPY) {
+            raw = earlier32(t.wA, a, lenA, e);
+            war = earlier32(t.rA, a, lenA, e);
+            waw = raw;
+            if (raw) mark_src(a);
+          } else if constexpr (OP == JP_OP_PRIV_TMP) {
+            war = earlier32(rT, a, lenT, e);
+            waw = earlier32(t.wT, a, lenT, e) || earlier32(t.wA, q4(vb[u], k), lenA, e);
+          } else {
+            const bool r0 = earlier32(t.wA, q4(vb[u], k), lenA, e), r1 = earlier32(t.wA, q4(vc[u], k), lenA, e);
+            raw = r0 || r1;
+            war = earlier32(t.rA, a, lenA, e);
+            waw = earlier32(t.wA, a, lenA, e);
+            if (r0) mark_src(q4(vb[u], k));
+            if (r1) mark_src(q4(vc[u], k));
+          }
+          c_raw += raw; c_war += war; c_waw += waw;
+          rb |= (uint32_t)raw << k;
+          if (raw && first == ~0ull) first = (unsigned long long)(L.base + (q << 2) + k);
         }
-        c_raw += raw; c_war += war; c_waw += waw;
-        if (raw && first == ~0ull) first = (unsigned long long)(L.base + (q << 2) + k);
+      }
+      if constexpr (GUIDE) {
+        // lanes 8m..8m+7 hold the 32 iterations of one word (q0 of lane 0 is a multiple of 8)
+        uint32_t wv = rb << (4 * (threadIdx.x & 7));
+        wv |= __shfl_xor_sync(0xffffffffu, wv, 1);
+        wv |= __shfl_xor_sync(0xffffffffu, wv, 2);
+        wv |= __shfl_xor_sync(0xffffffffu, wv, 4);
+        if ((threadIdx.x & 7) == 0 && q < nq) graw[q >> 3] = wv;
       }
     }
   }
@@ -450,7 +480,8 @@ static void run_classify(const DLoop &d, Tabs t, uint32_t *bits, int64_t chunk, 
   int64_t tiles = (d.n + 31) / 32;
   if (!bits && !cc) {
     const int64_t nq = (d.n + 3) / 4;
-    k_prof_count4<OP><<<grid_for((nq + kQuadSteps - 1) / kQuadSteps, 256, 8), 256, 0, st>>>(d, t, idx_vec(d), hdr);
+    k_prof_count4<OP, false><<<grid_for((nq + kQuadSteps - 1) / kQuadSteps, 256, 8), 256, 0, st>>>(d, t, idx_vec(d), hdr,
+                                                                                                 nullptr, nullptr);
   } else {
     k_prof_classify<OP><<<grid_for((tiles + kUnroll - 1) / kUnroll * 32, 256, 8), 256, 0, st>>>(d, t, bits, chunk, cc, hdr);
   }
@@ -466,6 +497,34 @@ cudaError_t launch_prof_classify(const Job &j, void *ws, const Layout &lo, uint3
   if (j.d.n == 0) return launch_check();
   Tabs t = tabs_of(j.d, ws, lo);
   JP_DISPATCH(j.op, j.dt, run_classify, j.d, t, raw_bits, chunk, chunk_counts, hdr, st);
+  return launch_check();
+}
+
+template <int OP, int DT>
+static void run_classify_guide(const DLoop &d, Tabs t, uint32_t *graw, uint32_t *gsrc, int64_t *hdr, cudaStream_t st) {
+  (void)DT;
+  const int64_t nq = (d.n + 3) / 4;
+  if constexpr (OP == JP_OP_PRIV_TMP) {   // never guided: counts only
+    k_prof_count4<OP, false><<<grid_for((nq + kQuadSteps - 1) / kQuadSteps, 256, 8), 256, 0, st>>>(d, t, idx_vec(d), hdr,
+                                                                                                 nullptr, nullptr);
+  } else {
+    k_prof_count4<OP, true><<<grid_for((nq + kQuadSteps - 1) / kQuadSteps, 256, 8), 256, 0, st>>>(d, t, idx_vec(d), hdr,
+                                                                                                graw, gsrc);
+  }
+  note_launch();
+}
+
+cudaError_t launch_prof_classify_guide(const Job &j, void *ws, const Layout &lo, cudaStream_t st) {
+  int64_t *hdr = at<int64_t>(ws, lo, R_HEADER);
+  uint32_t *bits = at<uint32_t>(ws, lo, R_GUIDE);
+  if (!bits) return launch_prof_classify(j, ws, lo, nullptr, 0, nullptr, st);
+  cudaMemsetAsync(&hdr[H_RAW], 0, 3 * sizeof(int64_t), st);
+  cudaMemsetAsync(&hdr[H_FIRST_RAW], 0xFF, sizeof(int64_t), st);
+  const int64_t nw = (j.d.n + 31) / 32;
+  cudaMemsetAsync(bits + nw, 0, 4 * (size_t)nw, st);   // source words are OR-ed in
+  if (j.d.n == 0) return launch_check();
+  Tabs t = tabs_of(j.d, ws, lo);
+  JP_DISPATCH(j.op, j.dt, run_classify_guide, j.d, t, bits, bits + nw, hdr, st);
   return launch_check();
 }
 

@@ -130,7 +130,7 @@ __device__ __forceinline__ uint32_t fwd_body(const DLoop &L, uint32_t a0, uint32
 
 template <int OP, int DT, bool GUIDED>
 __global__ void __launch_bounds__(kFwdThreads, 1)
-    k_tls_fwd(DLoop L, int track, int logC, uint32_t W, const uint32_t *gbits, int64_t *stats) {
+    k_tls_fwd(DLoop L, int track, int logC, uint32_t W, const uint32_t *graw, const uint32_t *gsrc, int64_t *stats) {
   constexpr int T = kFwdThreads, K = kFwdK;
   // ops whose exposed A read may hit another iteration's write: ADD_C A[r],
   // STENCIL2 A[r], A[r2].  SAXPY reads Y[w] (its own write address) and X;
@@ -147,7 +147,6 @@ __global__ void __launch_bounds__(kFwdThreads, 1)
   const uint32_t n32 = (uint32_t)L.n;
   const uint32_t io = (uint32_t)L.ioff;
   const bool trk = kTr && track;
-  const uint32_t nwords = (n32 + 31) >> 5;
   FwdLog H{smem_u32(fsm), kFwdHashLog + logC};
   const uint32_t ovbase = smem_u32(OV);
 
@@ -180,8 +179,8 @@ __global__ void __launch_bounds__(kFwdThreads, 1)
         if constexpr (OP == JP_OP_STENCIL2) R2[k] = L.r2 ? __ldg(L.r2 + i) : (int32_t)(io + i);
         if constexpr (OP == JP_OP_PRIV_TMP) R2[k] = L.s ? __ldg(L.s + i) : (int32_t)(io + i);
         if constexpr (GUIDED) {
-          bits |= ((__ldg(gbits + (i >> 5)) >> (i & 31)) & 1u) << k;
-          bits |= ((__ldg(gbits + nwords + (i >> 5)) >> (i & 31)) & 1u) << (K + k);
+          bits |= ((__ldg(graw + (i >> 5)) >> (i & 31)) & 1u) << k;
+          bits |= ((__ldg(gsrc + (i >> 5)) >> (i & 31)) & 1u) << (K + k);
         }
       }
     }
@@ -356,6 +355,263 @@ __global__ void __launch_bounds__(kFwdThreads, 1)
   }
 }
 
+// ---------------------------------------------------------------------------
+// grid path: every SM.  The window holds up to 2048 * CTAs iterations; the
+// write log is a stamp table S[a] = epoch << 32 | writer offset and the shadow
+// slots are V[a] = epoch << 32 | value, both in global memory (L2) and indexed
+// by ADDRESS (an address has at most one writer in the loop, so neither is
+// ever cleared: a stale epoch reads as "no writer in this window").  A reader
+// that finds an earlier in-window writer in S polls V at its own read address.
+// One software grid barrier per window (monotone counter, release/acquire).
+// ---------------------------------------------------------------------------
+__device__ __forceinline__ void fwd_grid_sync(unsigned *count, unsigned target) {
+  JP_CTA_SYNC();
+  if (threadIdx.x == 0) {
+    asm volatile("fence.acq_rel.gpu;\n\tred.relaxed.gpu.global.add.u32 [%0], 1;" ::"l"(count) : "memory");
+    unsigned v;
+    do {
+      asm volatile("ld.relaxed.gpu.global.u32 %0, [%1];" : "=r"(v) : "l"(count) : "memory");
+    } while (v < target);
+    asm volatile("fence.acq_rel.gpu;" ::: "memory");
+  }
+  JP_CTA_SYNC();
+}
+__device__ __forceinline__ unsigned long long g_ld_relaxed(const unsigned long long *p) {
+  unsigned long long v;
+  asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+  return v;
+}
+__device__ __forceinline__ void g_st_relaxed(unsigned long long *p, unsigned long long v) {
+  asm volatile("st.relaxed.gpu.global.u64 [%0], %1;" ::"l"(p), "l"(v) : "memory");
+}
+
+template <int OP, int DT, bool GUIDED>
+__global__ void __launch_bounds__(kFwdThreads, 1)
+    k_tls_fwd_grid(DLoop L, int track, uint32_t W, const uint32_t *graw, const uint32_t *gsrc, unsigned long long *S,
+                   unsigned long long *V, unsigned *bar, int64_t *stats) {
+  constexpr int T = kFwdThreads, K = kFwdK;
+  constexpr bool kTr = OP == JP_OP_ADD_C || OP == JP_OP_STENCIL2;
+  constexpr bool k2 = OP == JP_OP_STENCIL2;
+  const int tid = threadIdx.x;
+  const uint32_t G = gridDim.x * (uint32_t)T;
+  const uint32_t g = blockIdx.x * (uint32_t)T + (uint32_t)tid;
+  const uint32_t n32 = (uint32_t)L.n;
+  const uint32_t io = (uint32_t)L.ioff;
+  const bool trk = kTr && track;
+
+  int32_t cr[K], cw[K], c2[K], nr[K], nw[K], n2[K];
+  uint32_t cb = 0, nb = 0, g0[K], g1[K], ng0[K], ng1[K];
+  auto load_idx = [&](uint32_t ws, int32_t *R, int32_t *Wi, int32_t *R2, uint32_t &bits) {
+    bits = 0;
+#pragma unroll
+    for (int k = 0; k < K; k++) {
+      const uint32_t off = (uint32_t)k * G + g, i = ws + off;
+      if (off < W && i < n32) {
+        R[k] = L.r ? __ldg(L.r + i) : (int32_t)(io + i);
+        Wi[k] = L.w ? __ldg(L.w + i) : (int32_t)(io + i);
+        if constexpr (OP == JP_OP_STENCIL2) R2[k] = L.r2 ? __ldg(L.r2 + i) : (int32_t)(io + i);
+        if constexpr (OP == JP_OP_PRIV_TMP) R2[k] = L.s ? __ldg(L.s + i) : (int32_t)(io + i);
+        if constexpr (GUIDED) {
+          bits |= ((__ldg(graw + (i >> 5)) >> (i & 31)) & 1u) << k;
+          bits |= ((__ldg(gsrc + (i >> 5)) >> (i & 31)) & 1u) << (K + k);
+        }
+      }
+    }
+  };
+  auto gather = [&](uint32_t ws, const int32_t *R, const int32_t *Wi, const int32_t *R2, uint32_t *a0, uint32_t *a1) {
+#pragma unroll
+    for (int k = 0; k < K; k++) {
+      const uint32_t off = (uint32_t)k * G + g;
+      if (off < W && ws + off < n32) {
+        if constexpr (OP == JP_OP_ADD_C) a0[k] = __ldcg(L.A + R[k]);
+        else if constexpr (OP == JP_OP_SAXPY) { a0[k] = __ldg(L.X + R[k]); a1[k] = __ldcg(L.A + Wi[k]); }
+        else if constexpr (OP == JP_OP_PRIV_TMP) a0[k] = __ldg(L.X + R[k]);
+        else { a0[k] = __ldcg(L.A + R[k]); a1[k] = __ldcg(L.A + R2[k]); }
+      }
+    }
+  };
+
+  const uint32_t nwin = (n32 + W - 1) / W;
+  load_idx(0, cr, cw, c2, cb);
+  gather(0, cr, cw, c2, g0, g1);
+  if (nwin > 1) load_idx(W, nr, nw, n2, nb);
+  uint32_t viol = 0, dup = 0;
+  for (uint32_t win = 0; win < nwin; win++) {
+    const uint32_t ws = win * W, epoch = win + 1;
+    const unsigned long long tag = (unsigned long long)epoch << 32;
+    const bool more = win + 1 < nwin;
+    // ---------------- SE: log this window's writes (S[w] = epoch | offset) ----------------
+    unsigned long long old[K];
+#pragma unroll
+    for (int k = 0; k < K; k++) {
+      const uint32_t off = (uint32_t)k * G + g;
+      old[k] = 0;
+      bool log = trk && off < W && ws + off < n32;
+      if constexpr (GUIDED) log = log && ((cb >> (K + k)) & 1u);
+      if (log) old[k] = atomicExch(S + cw[k], tag | off);
+    }
+    fwd_grid_sync(bar, gridDim.x * (win + 1));
+#pragma unroll
+    for (int k = 0; k < K; k++) dup += (uint32_t)(old[k] >> 32) == epoch;   // a second writer in this window
+    if (more) gather(ws + W, nr, nw, n2, ng0, ng1);
+    // ---------------- DC ----------------
+    uint32_t pend = 0;   // bit k: operand 0 of slot k waits; bit K+k: operand 1
+#pragma unroll
+    for (int k = 0; k < K; k++) {
+      const uint32_t off = (uint32_t)k * G + g;
+      bool chk = trk && off < W && ws + off < n32;
+      if constexpr (GUIDED) chk = chk && ((cb >> k) & 1u);
+      if (chk) {
+        const unsigned long long s0 = __ldcg(S + cr[k]);
+        if ((s0 & ~0xFFFFFFFFull) == tag && (uint32_t)s0 < off) pend |= 1u << k;
+        if constexpr (k2) {
+          const unsigned long long s1 = __ldcg(S + c2[k]);
+          if ((s1 & ~0xFFFFFFFFull) == tag && (uint32_t)s1 < off) pend |= 1u << (K + k);
+        }
+      }
+    }
+    viol += __popc((pend | (pend >> K)) & ((1u << K) - 1));
+    // ---------------- non-violators: values, published where a later reader may wait ----------------
+    uint32_t va[K], vt[K];
+#pragma unroll
+    for (int k = 0; k < K; k++) {
+      const uint32_t off = (uint32_t)k * G + g;
+      const bool act = off < W && ws + off < n32;
+      if (act && !((pend >> k) & 1u) && !((pend >> (K + k)) & 1u)) {
+        va[k] = fwd_body<OP, DT>(L, g0[k], g1[k], vt[k]);
+        bool pub = trk;
+        if constexpr (GUIDED) pub = pub && ((cb >> (K + k)) & 1u);
+        if (pub) g_st_relaxed(V + cw[k], tag | va[k]);
+      }
+    }
+    // ---------------- recovery ----------------
+    while (__any_sync(0xffffffffu, pend)) {
+#pragma unroll
+      for (int k = 0; k < K; k++) {
+        if (((pend >> k) | (pend >> (K + k))) & 1u) {
+          if ((pend >> k) & 1u) {
+            const unsigned long long v = g_ld_relaxed(V + cr[k]);
+            if ((v & ~0xFFFFFFFFull) == tag) { g0[k] = (uint32_t)v; pend &= ~(1u << k); }
+          }
+          if constexpr (k2) {
+            if ((pend >> (K + k)) & 1u) {
+              const unsigned long long v = g_ld_relaxed(V + c2[k]);
+              if ((v & ~0xFFFFFFFFull) == tag) { g1[k] = (uint32_t)v; pend &= ~(1u << (K + k)); }
+            }
+          }
+          if (!(((pend >> k) | (pend >> (K + k))) & 1u)) {
+            va[k] = fwd_body<OP, DT>(L, g0[k], g1[k], vt[k]);
+            bool pub = true;
+            if constexpr (GUIDED) pub = (cb >> (K + k)) & 1u;
+            if (pub) g_st_relaxed(V + cw[k], tag | va[k]);
+          }
+        }
+      }
+    }
+    // ---------------- commit ----------------
+#pragma unroll
+    for (int k = 0; k < K; k++) {
+      const uint32_t off = (uint32_t)k * G + g;
+      if (off < W && ws + off < n32) {
+        __stcg(L.A + cw[k], va[k]);
+        if constexpr (OP == JP_OP_PRIV_TMP) __stcg(L.T + c2[k], vt[k]);
+      }
+    }
+    // ---------------- forward this window's writes into the next window's operands ----------------
+    uint32_t fx = 0, f0[K], f1[K];
+    if (more && trk) {
+#pragma unroll
+      for (int k = 0; k < K; k++) {
+        const uint32_t off = (uint32_t)k * G + g;
+        bool chk = off < W && ws + W + off < n32;
+        if constexpr (GUIDED) chk = chk && ((nb >> k) & 1u);
+        if (chk) {
+          if ((__ldcg(S + nr[k]) & ~0xFFFFFFFFull) == tag) {
+            unsigned long long v;
+            do { v = g_ld_relaxed(V + nr[k]); } while ((v & ~0xFFFFFFFFull) != tag);
+            f0[k] = (uint32_t)v;
+            fx |= 1u << k;
+          }
+          if constexpr (k2) {
+            if ((__ldcg(S + n2[k]) & ~0xFFFFFFFFull) == tag) {
+              unsigned long long v;
+              do { v = g_ld_relaxed(V + n2[k]); } while ((v & ~0xFFFFFFFFull) != tag);
+              f1[k] = (uint32_t)v;
+              fx |= 1u << (K + k);
+            }
+          }
+        }
+      }
+    }
+#pragma unroll
+    for (int k = 0; k < K; k++) {
+      cr[k] = nr[k]; cw[k] = nw[k];
+      if constexpr (OP == JP_OP_STENCIL2 || OP == JP_OP_PRIV_TMP) c2[k] = n2[k];
+      g0[k] = ((fx >> k) & 1u) ? f0[k] : ng0[k];
+      g1[k] = ((fx >> (K + k)) & 1u) ? f1[k] : ng1[k];
+    }
+    cb = nb;
+    if (win + 2 < nwin) load_idx(ws + 2 * W, nr, nw, n2, nb);
+  }
+  // ---------------- stats: stats[3] and the dup counter (bar[1]) were zeroed by the launcher ----------------
+  viol = __reduce_add_sync(0xffffffffu, viol);
+  dup = __reduce_add_sync(0xffffffffu, dup);
+  if ((tid & 31) == 0) {
+    if (viol) atomicAdd(reinterpret_cast<unsigned long long *>(&stats[3]), (unsigned long long)viol);
+    if (dup) atomicAdd(bar + 1, dup);
+  }
+  fwd_grid_sync(bar, gridDim.x * (nwin + 1));
+  if (blockIdx.x == 0 && tid == 0) {
+    const int64_t v = *(volatile int64_t *)&stats[3];
+    stats[0] = *(volatile unsigned *)(bar + 1) ? -1 : (int64_t)n32;
+    stats[1] = (int64_t)n32 + v;
+    stats[2] = nwin;
+  }
+}
+
+template <int OP, int DT>
+static void run_fwd_grid(cudaError_t &e, const Job &j, uint32_t W, const uint32_t *bits, const uint32_t *bsrc,
+                         unsigned long long *S,
+                         unsigned long long *V, unsigned *bar, int64_t *stats, cudaStream_t st) {
+  void *fn = bits ? (void *)k_tls_fwd_grid<OP, DT, true> : (void *)k_tls_fwd_grid<OP, DT, false>;
+  const int grid = (int)((W + kFwdThreads * kFwdK - 1) / (kFwdThreads * kFwdK));
+  int maxb = 0;
+  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&maxb, fn, kFwdThreads, 0);
+  if (grid > num_sms() * (maxb > 0 ? maxb : 1)) { e = cudaErrorInvalidConfiguration; return; }
+  DLoop d = j.d;
+  int track = a_indirect(j.op, j.d.r, j.d.r2, j.d.w) ? 1 : 0;
+  void *args[] = {&d, &track, &W, &bits, &bsrc, &S, &V, &bar, &stats};
+  e = cudaLaunchCooperativeKernel(fn, dim3(grid), dim3(kFwdThreads), args, 0, st);
+  note_launch();
+}
+
+cudaError_t launch_tls_fwd_grid(const Job &j, int64_t window, const uint32_t *bits, const uint32_t *bsrc,
+                                unsigned long long *S,
+                                unsigned long long *V, int64_t lenS, unsigned *bar, int64_t *stats,
+                                cudaStream_t st) {
+  if (j.d.n == 0) {
+    cudaMemsetAsync(stats, 0, 4 * sizeof(int64_t), st);
+    return launch_check();
+  }
+  if (S && lenS > 0) {   // epoch 0: no writer yet
+    cudaMemsetAsync(S, 0, 8 * (size_t)lenS, st);
+    cudaMemsetAsync(V, 0, 8 * (size_t)lenS, st);
+  }
+  cudaMemsetAsync(bar, 0, 2 * sizeof(unsigned), st);
+  cudaMemsetAsync(stats, 0, 4 * sizeof(int64_t), st);
+  cudaError_t e = cudaSuccess;
+  JP_DISPATCH(j.op, j.dt, run_fwd_grid, e, j, (uint32_t)window, bits, bsrc, S, V, bar, stats, st);
+  if (e != cudaSuccess) return e;
+  return launch_check();
+}
+
+int64_t tls_fwd_grid_wcap() {
+  int maxb = 0;
+  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&maxb, (void *)k_tls_fwd_grid<JP_OP_ADD_C, JP_I32, true>, kFwdThreads, 0);
+  cudaGetLastError();
+  return (int64_t)kFwdThreads * kFwdK * num_sms() * (maxb > 0 ? maxb : 1);
+}
+
 // Largest cluster (power of two <= 16) the device schedules for k_tls_fwd (cached per device).
 int tls_fwd_max_cluster() {
   static int cache[64] = {0};
@@ -386,8 +642,8 @@ int tls_fwd_max_cluster() {
 }
 
 template <int OP, int DT>
-static void run_fwd(cudaError_t &e, const Job &j, uint32_t W, int C, const uint32_t *bits, int64_t *stats,
-                    cudaStream_t st) {
+static void run_fwd(cudaError_t &e, const Job &j, uint32_t W, int C, const uint32_t *bits, const uint32_t *bsrc,
+                    int64_t *stats, cudaStream_t st) {
   int logC = 0;
   while ((1 << logC) < C) logC++;
   void *fn = bits ? (void *)k_tls_fwd<OP, DT, true> : (void *)k_tls_fwd<OP, DT, false>;
@@ -408,19 +664,19 @@ static void run_fwd(cudaError_t &e, const Job &j, uint32_t W, int C, const uint3
   cfg.numAttrs = 1;
   DLoop d = j.d;
   int track = a_indirect(j.op, j.d.r, j.d.r2, j.d.w) ? 1 : 0;
-  void *args[] = {&d, &track, &logC, &W, &bits, &stats};
+  void *args[] = {&d, &track, &logC, &W, &bits, &bsrc, &stats};
   e = cudaLaunchKernelExC(&cfg, fn, args);
   note_launch();
 }
 
-cudaError_t launch_tls_fwd(const Job &j, int64_t window, int cluster, const uint32_t *bits, int64_t *stats,
-                           cudaStream_t st) {
+cudaError_t launch_tls_fwd(const Job &j, int64_t window, int cluster, const uint32_t *bits, const uint32_t *bsrc,
+                           int64_t *stats, cudaStream_t st) {
   if (j.d.n == 0) {
     cudaMemsetAsync(stats, 0, 4 * sizeof(int64_t), st);
     return launch_check();
   }
   cudaError_t e = cudaSuccess;
-  JP_DISPATCH(j.op, j.dt, run_fwd, e, j, (uint32_t)window, cluster, bits, stats, st);
+  JP_DISPATCH(j.op, j.dt, run_fwd, e, j, (uint32_t)window, cluster, bits, bsrc, stats, st);
   if (e != cudaSuccess) return e;
   return launch_check();
 }

@@ -546,18 +546,31 @@ def test_schedule_modes_fig2b():
 
 
 @pytest.mark.parametrize("n,chunk", [(1 << 16, 1024), ((1 << 18), 4096)])
-def test_schedule_stealing_config5(n, chunk):
+@pytest.mark.parametrize("recovery", [0, 1])
+def test_schedule_stealing_config5(n, chunk, recovery):
+    """recovery 0 (auto): the write-once TLS task runs with on-chip recovery on a
+    cluster beside the partitioned tasks; 1: restart recovery on one SM."""
     wl = synth.config5(n=n)
-    _, A, T = O.run_seq(to_oracle(wl))
+    ref = to_oracle(wl)
+    _, A, T = O.run_seq(ref)
     g = gpu(wl)
     L = jp.Loop.from_workload(g)
-    res = jp.jp_schedule(L, jp.workspace(L), scheme=jp.JP_SCHED_STEALING, chunk_iters=chunk)
+    res = jp.jp_schedule(L, jp.workspace(L), scheme=jp.JP_SCHED_STEALING, chunk_iters=chunk, tls_recovery=recovery)
     torch.cuda.synchronize()
     check_arrays(g, A, T)
     assert res["task_mode_iters"][jp.JP_MODE_DOALL] == n // 2
     assert res["task_mode_iters"][jp.JP_MODE_TLS] == n // 4
     assert res["task_mode_iters"][jp.JP_MODE_PRIVATIZED] == n // 4
     assert res["n_batches"] == 1
+    b, e = n // 2, 3 * n // 4   # the TLS task, as a loop of its own
+    mid = O.Loop(ref.op, ref.dtype, e - b, ref.A, r=ref.r[b:e], w=ref.w[b:e], c0=ref.c0)
+    if recovery == 0:
+        assert res["tls_recovery"] == jp.JP_TLS_ONCHIP and res["tls_path"] == 5 and res["tls_guided"] == 1
+        assert res["tls"] == O.sim_tls_fwd(mid, res["tls_w_max"])[3]
+    else:
+        assert res["tls_recovery"] == jp.JP_TLS_RESTART and res["tls_path"] == 1
+        raw = O.profile(mid)["raw_iters"]
+        assert res["tls"] == O.sim_tls(mid, 0, res["tls_w_max"], raw)[3]
 
 
 def test_schedule_stealing_dependent_tasks():

@@ -33,9 +33,13 @@ def same(t: torch.Tensor, a: np.ndarray) -> bool:
     return t.cpu().numpy().tobytes() == a.tobytes()
 
 
-def fwd_case(wl, window, cluster=0, guided=False, view=None):
-    """Profile -> (guide) -> on-chip TLS; compare with the oracle.  window = 0:
-    the path's own window (2048 * cluster), returned by the check."""
+def grid_w():
+    return 2048 * torch.cuda.get_device_properties(0).multi_processor_count
+
+
+def fwd_case(wl, window, cluster=0, guided=False, view=None, path=5):
+    """Profile -> (guide) -> on-chip TLS on path 5 (cluster) or 6 (every SM);
+    compare with the oracle.  window = 0: the path's own window."""
     ref = to_oracle(wl)
     g = wl.to(DEV)
     L = jp.Loop.from_workload(g) if view is None else view(g)
@@ -45,10 +49,12 @@ def fwd_case(wl, window, cluster=0, guided=False, view=None):
     if guided:
         jp.jp_tls_guide(L, ws)
     got = jp.jp_run_tls(L, window=window, prof=p, ws=ws, cluster=cluster, guided=guided,
-                        recovery=jp.JP_TLS_ONCHIP)
+                        recovery=jp.JP_TLS_ONCHIP, path=path)
     torch.cuda.synchronize()
     W = window
-    if W == 0:
+    if W == 0 and path == 6:
+        W = grid_w()
+    elif W == 0:
         c = cluster
         if c == 0:
             c = 1
@@ -66,8 +72,9 @@ def fwd_case(wl, window, cluster=0, guided=False, view=None):
 
 @pytest.mark.parametrize("window", [1, 32, 100, 1000, 2048, 4096, 0])
 @pytest.mark.parametrize("d", [0.0, 0.05])
-def test_fwd_config1(window, d):
-    fwd_case(synth.config1(d), window)
+@pytest.mark.parametrize("path", [5, 6])
+def test_fwd_config1(window, d, path):
+    fwd_case(synth.config1(d), window, path=path)
 
 
 @pytest.mark.parametrize("cluster", [1, 2, 4, 8, 16])
@@ -84,6 +91,8 @@ def test_fwd_config3_reduced(d, guided):
     wl = synth.config3(d, n=(1 << 17) + 11)
     for window in (4096, 32768, 0):
         fwd_case(wl, window, guided=guided)
+    for window in (4096, 100000, 0):
+        fwd_case(wl, window, guided=guided, path=6)
 
 
 @pytest.mark.parametrize("op,dt", [(op, dt) for op in OPS for dt in DTS])
@@ -97,6 +106,10 @@ def test_fwd_random_write_once(op, dt):
         fwd_case(wl, window, cluster=cluster)
         if op != O.OP_PRIV_TMP:
             fwd_case(wl, window, cluster=cluster, guided=True)
+    for window in (64, 2500, 0):
+        fwd_case(wl, window, path=6)
+        if op != O.OP_PRIV_TMP:
+            fwd_case(wl, window, guided=True, path=6)
 
 
 def test_fwd_chains():
@@ -114,6 +127,9 @@ def test_fwd_chains():
     for window in (777, 32768):
         fwd_case(gs, window)
         fwd_case(gs, window, guided=True)
+    for window in (1000, 40000):
+        assert fwd_case(pc, window, path=6)["violations"] == n - -(-n // window)
+        fwd_case(gs, window, path=6, guided=True)
 
 
 def test_fwd_unaligned_views():
@@ -147,7 +163,8 @@ def test_fwd_repeatability():
     jp.jp_tls_guide(L, ws)
     for rep in range(10):
         g.A.copy_(A0)
-        got = jp.jp_run_tls(L, window=32768, prof=p, ws=ws, guided=bool(rep & 1), recovery=jp.JP_TLS_ONCHIP)
+        got = jp.jp_run_tls(L, window=32768, prof=p, ws=ws, guided=bool(rep & 1), recovery=jp.JP_TLS_ONCHIP,
+                            path=5 + (rep & 2) // 2)
         torch.cuda.synchronize()
         assert same(g.A, A) and got == stats, rep
 
@@ -167,7 +184,7 @@ def test_fwd_needs_write_once_profile():
     L3 = jp.Loop.from_workload(wl3)
     p3 = jp.jp_profile_density(L3, jp.workspace(L3))
     with pytest.raises(jp.JPError):          # window larger than a 16-CTA cluster holds
-        jp.jp_run_tls(L3, window=2048 * 16 + 1, prof=p3, ws=jp.workspace(L3), recovery=jp.JP_TLS_ONCHIP)
+        jp.jp_run_tls(L3, window=2048 * 16 + 1, prof=p3, ws=jp.workspace(L3), recovery=jp.JP_TLS_ONCHIP, path=5)
     with pytest.raises(jp.JPError):          # window larger than the given cluster holds
         jp.jp_run_tls(L3, window=4097, cluster=2, prof=p3, ws=jp.workspace(L3), recovery=jp.JP_TLS_ONCHIP)
 
@@ -182,8 +199,50 @@ def test_fwd_config3_full_size_schedule(d):
     L = jp.Loop.from_workload(g)
     res = jp.jp_schedule(L, jp.workspace(L))
     torch.cuda.synchronize()
-    assert res["mode"] == jp.JP_MODE_TLS and res["tls_recovery"] == jp.JP_TLS_ONCHIP and res["tls_path"] == 5
-    assert res["tls_cluster"] == 16 and res["tls_w_max"] == 32768
+    assert res["mode"] == jp.JP_MODE_TLS and res["tls_recovery"] == jp.JP_TLS_ONCHIP and res["tls_path"] == 6
+    assert res["tls_w_max"] == grid_w() and res["tls_guided"] == 1
     _, A, _, stats = O.sim_tls_fwd(ref, res["tls_w_max"])
     assert same(g.A, A)
     assert res["tls"] == stats, (res["tls"], stats)
+
+
+def test_fwd_grid_window_cap():
+    wl = synth.config3(0.01, n=1 << 16).to(DEV)
+    L = jp.Loop.from_workload(wl)
+    ws = jp.workspace(L)
+    p = jp.jp_profile_density(L, ws)
+    with pytest.raises(jp.JPError):
+        jp.jp_run_tls(L, window=grid_w() + 1, prof=p, ws=ws, recovery=jp.JP_TLS_ONCHIP, path=6)
+    with pytest.raises(jp.JPError):          # not an on-chip path
+        jp.jp_run_tls(L, window=100, prof=p, ws=ws, recovery=jp.JP_TLS_ONCHIP, path=1)
+
+
+@pytest.mark.parametrize("case", ["c3_0", "c3_1", "c3_10", "stencil", "saxpy_null"])
+def test_schedule_fused_guide_bits(case):
+    """jp_schedule writes the guide bitmaps in its classify pass (no jp_tls_guide):
+    raw words == the oracle's raw flags, source words == oracle raw_sources, for
+    write-once loops (the only loops a guided run accepts); the run is exact."""
+    from helpers import bits_to_flags
+    if case.startswith("c3"):
+        wl = synth.config3({"c3_0": 0.0, "c3_1": 0.01, "c3_10": 0.10}[case], n=(1 << 16) + 9)
+    elif case == "stencil":
+        wl = random_loop(77, O.OP_STENCIL2, O.F32, 5000, len_a=15000, null_prob=0.0, dup_writes=False)
+    else:
+        wl = random_loop(78, O.OP_ADD_C, O.I32, 5003, len_a=15000, null_prob=0.5, dup_writes=False)
+    ref = to_oracle(wl)
+    _, A, _ = O.run_seq(ref)
+    g = wl.to(DEV)
+    L = jp.Loop.from_workload(g)
+    ws = jp.workspace(L)
+    res = jp.jp_schedule(L, ws)
+    torch.cuda.synchronize()
+    assert same(g.A, A)
+    off, nb = jp.jp_ws_region(L, "guide")
+    if nb == 0:
+        return
+    nw = (wl.n + 31) // 32
+    words = ws[off:off + 8 * nw].view(torch.int32)
+    assert np.array_equal(bits_to_flags(words[:nw], wl.n), O.profile(ref)["flags"] & 1)
+    assert np.array_equal(bits_to_flags(words[nw:], wl.n), O.raw_sources(ref))
+    if res["mode"] == jp.JP_MODE_TLS:
+        assert res["tls"] == O.sim_tls_fwd(ref, res["tls_w_max"])[3]
