@@ -936,7 +936,7 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
     Layout lo;
     JP_TRY(check_ws(L, ws, ws_bytes, 0, lo));
     int64_t *hdr = at<int64_t>(ws, lo, R_HEADER);
-    JP_CUDA(launch_tiny(j, L, c.tau_high, c.tls_window, c.tls_w_max, hdr, st), "tiny");
+    JP_CUDA(launch_tiny(j, L, c.tau_high, c.tls_window, c.tls_w_max, c.tls_recovery, hdr, st), "tiny");
     int64_t h[16];
     JP_CUDA(d2h_small_sync(h, hdr, sizeof h, st), "tiny D2H");
     if (h[H_TINY_MODE] < 0) return fail(JP_ERR_INDEX, "%lld index entries are outside their arrays", (long long)h[H_BAD]);
@@ -954,6 +954,8 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
       res->tls.violations = h[H_TLS_VIOL];
       res->tls_w_max = h[H_TINY_WMAX];
       res->tls_path = 4;
+      res->tls_recovery = (int32_t)h[H_TINY_REC];
+      res->tls_cluster = 1;
     }
     return JP_OK;
   }

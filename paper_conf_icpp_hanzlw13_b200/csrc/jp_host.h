@@ -71,8 +71,8 @@ cudaError_t launch_task_conflicts(const Job &j, const int32_t *chunk_task, int64
 
 // tiny loops (jp_tiny.cu): the whole schedule in one CTA's shared memory
 bool tiny_eligible(const jp_loop *L);
-cudaError_t launch_tiny(const Job &j, const jp_loop *L, double tau, int64_t window, int64_t w_max, int64_t *hdr,
-                        cudaStream_t st);
+cudaError_t launch_tiny(const Job &j, const jp_loop *L, double tau, int64_t window, int64_t w_max, int recovery,
+                        int64_t *hdr, cudaStream_t st);
 
 struct TlsPlan {
   int64_t window, w_max, prof_raw;  // prof_raw < 0: no profile

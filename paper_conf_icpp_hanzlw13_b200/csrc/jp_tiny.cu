@@ -25,6 +25,7 @@ constexpr uint32_t kTinyEpochs = 0xFFFFF;        // 20-bit window counter (windo
 struct TinyArgs {
   double tau;
   int64_t window, w_max;   // w_max 0: from the profiled density (as jp_schedule)
+  int recovery;            // jp_sched_cfg.tls_recovery: 0 auto (on chip when no address is written twice), 1 restart
 };
 
 template <int OP> __host__ __device__ constexpr int tiny_streams() { return (OP == JP_OP_PRIV_TMP || OP == JP_OP_STENCIL2) ? 3 : 2; }
@@ -56,6 +57,7 @@ __global__ void __launch_bounds__(kTinyThreads, 1) k_tiny(DLoop L, TinyArgs a, i
   uint32_t *sT = sA + lenA;                        // T values
   uint32_t *tA0 = sT + lenT, *tA1 = tA0 + lenA;    // per-address tables of A
   uint32_t *tT0 = tA1 + lenA, *tT1 = tT0 + lenT;   // per-address tables of T
+  uint32_t *rdy = tT1 + lenT;                      // on-chip TLS: window tag of the shadow value tA1[a]
   __shared__ unsigned s_cnt[4];                    // raw, war, waw, bad
   __shared__ int s_first, s_fv[2];
   const int tid = threadIdx.x, wbase = tid & ~31;
@@ -143,7 +145,102 @@ __global__ void __launch_bounds__(kTinyThreads, 1) k_tiny(DLoop L, TinyArgs a, i
                    : (war_n > 0 || waw_n > 0) ? JP_MODE_PRIVATIZED : JP_MODE_DOALL;
   long long committed = 0, executed = 0, windows = 0, viol = 0;
   int64_t wmax_used = 0;
-  if (mode == JP_MODE_DOALL) {
+  const bool onchip = mode != JP_MODE_DOALL && mode != JP_MODE_PRIVATIZED && waw_n == 0 && a.recovery != 1;
+  if (onchip) {
+    // ---- TLS with on-chip recovery (reading B7): fixed windows, every violator
+    // re-executed once with its operand forwarded from the writer's shadow slot.
+    // No address is written twice, so the window's write log is the first-writer
+    // table tA0 of the profile restricted to the window: the writer of an exposed
+    // read a is j = tA0[a], in the window iff ws <= j, earlier iff j < i.
+    // Shadow values live per address (tA1[a], tagged by rdy[a] = window + 1).
+    const int W = a.window > 0 ? (int)a.window : n;
+    wmax_used = W;
+    for (int e = tid; e < lenA; e += T) rdy[e] = 0;
+    JP_CTA_SYNC();
+    for (int ws = 0; ws < n; ws += W) {
+      const int span = min(W, n - ws);
+      const uint32_t tag = (uint32_t)windows + 1;
+      uint32_t va[K], vt[K], g0[K], g1[K];
+      uint32_t pend = 0;   // bit k: operand 0 waits on its writer; bit 16 + k: operand 1
+      unsigned nv = 0;
+      // SE from committed memory (sA) + DC against the window's writers
+#pragma unroll
+      for (int k = 0; k < K; k++) {
+        if (k * T + wbase >= span) break;   // warp-uniform
+        const int off = k * T + tid;
+        if (off < span) {
+          const int i = ws + off;
+          const int32_t r = ix[i], w = ix[n + i], x2 = NS == 3 ? ix[2 * n + i] : 0;
+          auto inwin = [&](int32_t addr) { const uint32_t j = tA0[addr]; return j >= (uint32_t)ws && j < (uint32_t)i; };
+          if constexpr (OP == JP_OP_ADD_C) { g0[k] = sA[r]; if (inwin(r)) pend |= 1u << k; }
+          else if constexpr (OP == JP_OP_SAXPY) { g0[k] = L.X[r]; g1[k] = sA[w]; }
+          else if constexpr (OP == JP_OP_PRIV_TMP) g0[k] = L.X[r];
+          else {
+            g0[k] = sA[r]; g1[k] = sA[x2];
+            if (inwin(r)) pend |= 1u << k;
+            if (inwin(x2)) pend |= 1u << (16 + k);
+          }
+          nv += ((pend >> k) | (pend >> (16 + k))) & 1u;
+        }
+      }
+      auto body = [&](int k) {
+        if constexpr (OP == JP_OP_ADD_C) va[k] = op_add<DT>(g0[k], L.c0);
+        else if constexpr (OP == JP_OP_SAXPY) va[k] = op_add<DT>(op_mul<DT>(L.c0, g0[k]), g1[k]);
+        else if constexpr (OP == JP_OP_PRIV_TMP) { vt[k] = op_mul<DT>(L.c0, g0[k]); va[k] = op_add<DT>(vt[k], L.c1); }
+        else va[k] = op_mul<DT>(op_add<DT>(g0[k], g1[k]), L.c0);
+      };
+      auto publish = [&](int k, int i) {
+        const int32_t w = ix[n + i];
+        *(volatile uint32_t *)&tA1[w] = va[k];
+        __threadfence_block();
+        *(volatile uint32_t *)&rdy[w] = tag;
+      };
+#pragma unroll
+      for (int k = 0; k < K; k++) {
+        if (k * T + wbase >= span) break;
+        const int off = k * T + tid;
+        if (off < span && !(((pend >> k) | (pend >> (16 + k))) & 1u)) { body(k); publish(k, ws + off); }
+      }
+      // recovery: violators in dependence order (their writers are earlier, so every wait ends)
+      while (__any_sync(0xffffffffu, pend)) {
+#pragma unroll
+        for (int k = 0; k < K; k++) {
+          if (((pend >> k) | (pend >> (16 + k))) & 1u) {
+            const int i = ws + k * T + tid;
+            if ((pend >> k) & 1u) {
+              const int32_t r = ix[i];
+              if (*(volatile uint32_t *)&rdy[r] == tag) { __threadfence_block(); g0[k] = *(volatile uint32_t *)&tA1[r]; pend &= ~(1u << k); }
+            }
+            if constexpr (OP == JP_OP_STENCIL2) {
+              if ((pend >> (16 + k)) & 1u) {
+                const int32_t x2 = ix[2 * n + i];
+                if (*(volatile uint32_t *)&rdy[x2] == tag) { __threadfence_block(); g1[k] = *(volatile uint32_t *)&tA1[x2]; pend &= ~(1u << (16 + k)); }
+              }
+            }
+            if (!(((pend >> k) | (pend >> (16 + k))) & 1u)) { body(k); publish(k, i); }
+          }
+        }
+      }
+      JP_CTA_SYNC();   // every read of committed memory in this window is done
+#pragma unroll
+      for (int k = 0; k < K; k++) {
+        if (k * T + wbase >= span) break;
+        const int off = k * T + tid;
+        if (off < span) {
+          const int i = ws + off;
+          sA[ix[n + i]] = va[k];
+          if constexpr (OP == JP_OP_PRIV_TMP) sT[ix[2 * n + i]] = vt[k];
+        }
+      }
+      nv = __reduce_add_sync(0xffffffffu, nv);
+      if ((tid & 31) == 0 && nv) atomicAdd(&s_cnt[3], nv);   // s_cnt[3] (bad) is 0 here: reused as the counter
+      JP_CTA_SYNC();   // commits visible to the next window
+      windows++;
+    }
+    viol = s_cnt[3];
+    committed = n;
+    executed = n + viol;
+  } else if (mode == JP_MODE_DOALL) {
     // ---- DOALL: no dependence, any order ----
     for (int i = tid; i < n; i += T) {
       const int32_t r = ix[i], w = ix[n + i], x2 = NS == 3 ? ix[2 * n + i] : 0;
@@ -297,13 +394,14 @@ __global__ void __launch_bounds__(kTinyThreads, 1) k_tiny(DLoop L, TinyArgs a, i
     hdr[H_TLS_WINDOWS] = windows; hdr[H_TLS_VIOL] = viol;
     hdr[H_TINY_MODE] = mode;
     hdr[H_TINY_WMAX] = wmax_used;
+    hdr[H_TINY_REC] = onchip ? JP_TLS_ONCHIP : JP_TLS_RESTART;
   }
 }
 
 size_t tiny_smem_bytes(const jp_loop *L) {
   const int ns = (L->op == JP_OP_PRIV_TMP || L->op == JP_OP_STENCIL2) ? 3 : 2;
   const int64_t lt = L->op == JP_OP_PRIV_TMP ? L->len_T : 0;
-  return (size_t)4 * ((size_t)ns * L->n + 3 * (size_t)L->len_A + 3 * (size_t)lt);
+  return (size_t)4 * ((size_t)ns * L->n + 4 * (size_t)L->len_A + 3 * (size_t)lt);
 }
 
 bool tiny_eligible(const jp_loop *L) {
@@ -332,12 +430,13 @@ static void run_tiny_v(cudaError_t &e, const DLoop &d, TinyArgs a, size_t smem, 
   e = run_tiny<OP, DT>(d, a, smem, hdr, st);
 }
 
-cudaError_t launch_tiny(const Job &j, const jp_loop *L, double tau, int64_t window, int64_t w_max, int64_t *hdr,
-                        cudaStream_t st) {
+cudaError_t launch_tiny(const Job &j, const jp_loop *L, double tau, int64_t window, int64_t w_max, int recovery,
+                        int64_t *hdr, cudaStream_t st) {
   TinyArgs a;
   a.tau = tau;
   a.window = window;
   a.w_max = w_max;
+  a.recovery = recovery;
   cudaError_t e = cudaSuccess;
   JP_DISPATCH(j.op, j.dt, run_tiny_v, e, j.d, a, tiny_smem_bytes(L), hdr, st);
   return e;

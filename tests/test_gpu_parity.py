@@ -638,14 +638,16 @@ def test_tls_cta_repeatability(waw):
 # ---------------------------------------------------------------------------
 # tiny loops: the whole schedule in one CTA (jp_tiny.cu)
 # ---------------------------------------------------------------------------
-def tiny_case(wl, expect_mode=None):
+def tiny_case(wl, expect_mode=None, **kw):
+    """kw: jp_sched_cfg fields (tls_recovery: 0 auto = on chip for write-once
+    loops, 1 restart; tls_window)."""
     ref = to_oracle(wl)
     _, A, T = O.run_seq(ref)
     p = O.profile(ref)
     g = gpu(wl)
     L = jp.Loop.from_workload(g)
     n0 = jp.jp_launch_count()
-    res = jp.jp_schedule(L, jp.workspace(L))
+    res = jp.jp_schedule(L, jp.workspace(L), **kw)
     torch.cuda.synchronize()
     assert jp.jp_launch_count() == n0 + 1           # one launch does profile + mode + run
     check_arrays(g, A, T)
@@ -655,7 +657,14 @@ def tiny_case(wl, expect_mode=None):
         assert res["mode"] == expect_mode
     if res["mode"] in (jp.JP_MODE_TLS, jp.JP_MODE_SEQ_RECOMMENDED):
         assert res["tls_path"] == 4
-        _, A2, _, stats = O.sim_tls(ref, 0, res["tls_w_max"], p["raw_iters"])
+        onchip = p["waw_iters"] == 0 and kw.get("tls_recovery", 0) != 1
+        assert res["tls_recovery"] == (jp.JP_TLS_ONCHIP if onchip else jp.JP_TLS_RESTART)
+        if onchip:
+            stats = O.sim_tls_fwd(ref, res["tls_w_max"])[3]
+        elif kw.get("tls_window", 0) > 0:
+            stats = O.sim_tls(ref, kw["tls_window"])[3]
+        else:
+            stats = O.sim_tls(ref, 0, res["tls_w_max"], p["raw_iters"])[3]
         assert res["tls"] == stats, (res["tls"], stats)
     return res
 
@@ -705,3 +714,13 @@ def test_tiny_bad_index_no_side_effects():
     assert e.value.status == -5
     torch.cuda.synchronize()
     assert torch.equal(g.A, A0)
+
+
+@pytest.mark.parametrize("kw", [dict(tls_recovery=1), dict(tls_window=100), dict(tls_window=100, tls_recovery=1),
+                                dict(tls_window=1)])
+def test_tiny_recovery_and_windows(kw):
+    """The one-CTA schedule with on-chip recovery (fixed windows) and with restart recovery."""
+    res = tiny_case(synth.config1(0.05), jp.JP_MODE_TLS, **kw)
+    if kw.get("tls_window"):
+        assert res["tls"]["windows"] >= -(-4096 // kw["tls_window"])
+    tiny_case(random_loop(41, O.OP_STENCIL2, O.F32, 3000, len_a=6000, null_prob=0.0, dup_writes=False), **kw)
