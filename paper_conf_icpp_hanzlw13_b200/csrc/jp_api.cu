@@ -573,6 +573,7 @@ jp_status jp_run_tls(const jp_loop *L, const jp_tls_cfg *cfg, const jp_profile *
 
 #ifdef JP_TLS_TRACE
 int32_t jp_tls_trace(long long *host, int32_t n) { return (int32_t)jp::tls_trace_copy(host, n); }
+int32_t jp_tls_fwd_trace(long long *host, int32_t n) { return (int32_t)jp::tls_fwd_trace_copy(host, n); }
 #endif
 
 jp_status jp_merge_apply(void *arr, int64_t len, const int64_t *keys, jp_stream_t st) {

@@ -104,6 +104,7 @@ int64_t tls_cta_wcap(int op, bool waw, bool guided);   // largest single-CTA win
 int tls_max_cluster();                                 // 16 when the device schedules it, else 8
 #ifdef JP_TLS_TRACE
 cudaError_t tls_trace_copy(long long *host, int n);
+cudaError_t tls_fwd_trace_copy(long long *host, int n);
 #endif
 
 }  // namespace jp

@@ -385,187 +385,252 @@ __device__ __forceinline__ void g_st_relaxed(unsigned long long *p, unsigned lon
   asm volatile("st.relaxed.gpu.global.u64 [%0], %1;" ::"l"(p), "l"(v) : "memory");
 }
 
-template <int OP, int DT, bool GUIDED>
-__global__ void __launch_bounds__(kFwdThreads, 1)
-    k_tls_fwd_grid(DLoop L, int track, uint32_t W, const uint32_t *graw, const uint32_t *gsrc, unsigned long long *S,
-                   unsigned long long *V, unsigned *bar, int64_t *stats) {
-  constexpr int T = kFwdThreads, K = kFwdK;
-  constexpr bool kTr = OP == JP_OP_ADD_C || OP == JP_OP_STENCIL2;
-  constexpr bool k2 = OP == JP_OP_STENCIL2;
-  const int tid = threadIdx.x;
-  const uint32_t G = gridDim.x * (uint32_t)T;
-  const uint32_t g = blockIdx.x * (uint32_t)T + (uint32_t)tid;
-  const uint32_t n32 = (uint32_t)L.n;
-  const uint32_t io = (uint32_t)L.ioff;
-  const bool trk = kTr && track;
+// Per-window state of one thread: the indices, guide bits and operands of its
+// K slots.  The kernel keeps two of these and alternates them (a two-window
+// unrolled loop), so loads issued for the next window land in registers that
+// are not touched again until that window runs: no register copy ever waits
+// on an outstanding load.
+template <int K>
+struct FwdSet {
+  int32_t r[K], w[K], x[K];   // read / write / (r2 | s) addresses
+  uint32_t g0[K], g1[K];      // operands (window-start values, patched by forwarding)
+  uint32_t gr[K], gs[K];      // guide words holding the slot's raw-reader / RAW-source bit (read
+                              // where the bit is used, so the loads never stall the index prefetch)
+};
 
-  int32_t cr[K], cw[K], c2[K], nr[K], nw[K], n2[K];
-  uint32_t cb = 0, nb = 0, g0[K], g1[K], ng0[K], ng1[K];
-  auto load_idx = [&](uint32_t ws, int32_t *R, int32_t *Wi, int32_t *R2, uint32_t &bits) {
-    bits = 0;
-#pragma unroll
-    for (int k = 0; k < K; k++) {
-      const uint32_t off = (uint32_t)k * G + g, i = ws + off;
-      if (off < W && i < n32) {
-        R[k] = L.r ? __ldg(L.r + i) : (int32_t)(io + i);
-        Wi[k] = L.w ? __ldg(L.w + i) : (int32_t)(io + i);
-        if constexpr (OP == JP_OP_STENCIL2) R2[k] = L.r2 ? __ldg(L.r2 + i) : (int32_t)(io + i);
-        if constexpr (OP == JP_OP_PRIV_TMP) R2[k] = L.s ? __ldg(L.s + i) : (int32_t)(io + i);
-        if constexpr (GUIDED) {
-          bits |= ((__ldg(graw + (i >> 5)) >> (i & 31)) & 1u) << k;
-          bits |= ((__ldg(gsrc + (i >> 5)) >> (i & 31)) & 1u) << (K + k);
-        }
-      }
-    }
-  };
-  auto gather = [&](uint32_t ws, const int32_t *R, const int32_t *Wi, const int32_t *R2, uint32_t *a0, uint32_t *a1) {
-#pragma unroll
-    for (int k = 0; k < K; k++) {
-      const uint32_t off = (uint32_t)k * G + g;
-      if (off < W && ws + off < n32) {
-        if constexpr (OP == JP_OP_ADD_C) a0[k] = __ldcg(L.A + R[k]);
-        else if constexpr (OP == JP_OP_SAXPY) { a0[k] = __ldg(L.X + R[k]); a1[k] = __ldcg(L.A + Wi[k]); }
-        else if constexpr (OP == JP_OP_PRIV_TMP) a0[k] = __ldg(L.X + R[k]);
-        else { a0[k] = __ldcg(L.A + R[k]); a1[k] = __ldcg(L.A + R2[k]); }
-      }
-    }
-  };
+#ifdef JP_TLS_TRACE
+// phase marks (SM clock) of CTA 0 / thread 0 per window (trace build only, scripts/tls_fwd_trace.py)
+__device__ long long g_fwd_trace[2048 * 16];
+cudaError_t tls_fwd_trace_copy(long long *host, int n) {
+  return cudaMemcpyFromSymbol(host, g_fwd_trace, sizeof(long long) * (size_t)n);
+}
+#define FTR(ph) do { if (blockIdx.x == 0 && threadIdx.x == 0 && win < 2048u) g_fwd_trace[win * 16 + (ph)] = clock64(); } while (0)
+#else
+#define FTR(ph) do { } while (0)
+#endif
 
-  const uint32_t nwin = (n32 + W - 1) / W;
-  load_idx(0, cr, cw, c2, cb);
-  gather(0, cr, cw, c2, g0, g1);
-  if (nwin > 1) load_idx(W, nr, nw, n2, nb);
+template <int OP, int DT, bool GUIDED, int K>
+struct FwdGrid {
+  static constexpr bool kTr = OP == JP_OP_ADD_C || OP == JP_OP_STENCIL2;
+  static constexpr bool k2 = OP == JP_OP_STENCIL2;
+  static constexpr int T = kFwdThreads;
+  DLoop L;
+  const uint32_t *graw, *gsrc;
+  unsigned long long *S, *V;
+  unsigned *bar;
+  uint32_t W, G, g, n32, io, nwin;
+  bool trk;
   uint32_t viol = 0, dup = 0;
-  for (uint32_t win = 0; win < nwin; win++) {
+
+  __device__ __forceinline__ bool act(uint32_t ws, int k) const {
+    const uint32_t off = (uint32_t)k * G + g;
+    return off < W && ws + off < n32;
+  }
+  __device__ __forceinline__ void load_idx(uint32_t ws, FwdSet<K> &s) const {
+#pragma unroll
+    for (int k = 0; k < K; k++) {
+      if (!act(ws, k)) continue;
+      // streamed once: evict-first, so that the gathered array stays in L2
+      const uint32_t i = ws + (uint32_t)k * G + g;
+      s.r[k] = L.r ? __ldcs(L.r + i) : (int32_t)(io + i);
+      s.w[k] = L.w ? __ldcs(L.w + i) : (int32_t)(io + i);
+      if constexpr (OP == JP_OP_STENCIL2) s.x[k] = L.r2 ? __ldcs(L.r2 + i) : (int32_t)(io + i);
+      if constexpr (OP == JP_OP_PRIV_TMP) s.x[k] = L.s ? __ldcs(L.s + i) : (int32_t)(io + i);
+      if constexpr (GUIDED) {
+        s.gr[k] = __ldcs(graw + (i >> 5));
+        s.gs[k] = __ldcs(gsrc + (i >> 5));
+      }
+    }
+  }
+  // gathers of a window's operands; skip: bit k = operand 0 of slot k already
+  // forwarded, bit K+k = operand 1
+  __device__ __forceinline__ void gather(uint32_t ws, FwdSet<K> &s, uint32_t skip = 0) const {
+#pragma unroll
+    for (int k = 0; k < K; k++) {
+      if (!act(ws, k)) continue;
+      const bool s0 = (skip >> k) & 1u, s1 = (skip >> (K + k)) & 1u;
+      if constexpr (OP == JP_OP_ADD_C) { if (!s0) s.g0[k] = __ldcg(L.A + s.r[k]); }
+      else if constexpr (OP == JP_OP_SAXPY) { s.g0[k] = __ldg(L.X + s.r[k]); s.g1[k] = __ldcg(L.A + s.w[k]); }
+      else if constexpr (OP == JP_OP_PRIV_TMP) s.g0[k] = __ldg(L.X + s.r[k]);
+      else { if (!s0) s.g0[k] = __ldcg(L.A + s.r[k]); if (!s1) s.g1[k] = __ldcg(L.A + s.x[k]); }
+    }
+  }
+  // guide bits of slot k of the window starting at ws (true when unguided)
+  __device__ __forceinline__ bool raw_bit(const FwdSet<K> &s, uint32_t ws, int k) const {
+    if constexpr (GUIDED) return (s.gr[k] >> ((ws + (uint32_t)k * G + g) & 31)) & 1u;
+    else return true;
+  }
+  __device__ __forceinline__ bool src_bit(const FwdSet<K> &s, uint32_t ws, int k) const {
+    if constexpr (GUIDED) return (s.gs[k] >> ((ws + (uint32_t)k * G + g) & 31)) & 1u;
+    else return true;
+  }
+  static __device__ __forceinline__ bool cur(unsigned long long v, unsigned long long tag) {
+    return (v & ~0xFFFFFFFFull) == tag;
+  }
+
+  // one window: c = this window's set (indices, operands), nx = the next window's
+  // set (indices loaded; its gathers are issued here; its indices for the window
+  // after it are loaded into c at the end)
+  __device__ __forceinline__ void step(uint32_t win, FwdSet<K> &c, FwdSet<K> &nx) {
     const uint32_t ws = win * W, epoch = win + 1;
     const unsigned long long tag = (unsigned long long)epoch << 32;
     const bool more = win + 1 < nwin;
+    FTR(0);
     // ---------------- SE: log this window's writes (S[w] = epoch | offset) ----------------
     unsigned long long old[K];
 #pragma unroll
     for (int k = 0; k < K; k++) {
-      const uint32_t off = (uint32_t)k * G + g;
       old[k] = 0;
-      bool log = trk && off < W && ws + off < n32;
-      if constexpr (GUIDED) log = log && ((cb >> (K + k)) & 1u);
-      if (log) old[k] = atomicExch(S + cw[k], tag | off);
+      if (trk && act(ws, k) && src_bit(c, ws, k)) old[k] = atomicExch(S + c.w[k], tag | ((uint32_t)k * G + g));
     }
-    fwd_grid_sync(bar, gridDim.x * (win + 1));
+    FTR(1);
+    fwd_grid_sync(bar, gridDim.x * epoch);
+    FTR(2);
 #pragma unroll
     for (int k = 0; k < K; k++) dup += (uint32_t)(old[k] >> 32) == epoch;   // a second writer in this window
-    if (more) gather(ws + W, nr, nw, n2, ng0, ng1);
+    // ---------------- this window's DC probes and the next window's forwarding
+    // probes, all at once; the next window's gathers wait for the end of the
+    // window so that probes and polls do not queue behind them ----------------
+    unsigned long long p0[K], p1[K], q0[K], q1[K];
+#pragma unroll
+    for (int k = 0; k < K; k++) {
+      p0[k] = p1[k] = q0[k] = q1[k] = 0;
+      if (trk && act(ws, k) && raw_bit(c, ws, k)) {
+        p0[k] = __ldcg(S + c.r[k]);
+        if constexpr (k2) p1[k] = __ldcg(S + c.x[k]);
+      }
+      if (trk && more && act(ws + W, k) && raw_bit(nx, ws + W, k)) {
+        q0[k] = __ldcg(S + nx.r[k]);
+        if constexpr (k2) q1[k] = __ldcg(S + nx.x[k]);
+      }
+    }
     // ---------------- DC ----------------
-    uint32_t pend = 0;   // bit k: operand 0 of slot k waits; bit K+k: operand 1
+    uint32_t pend = 0;   // bit k: operand 0 of slot k waits for its writer; bit K+k: operand 1
 #pragma unroll
     for (int k = 0; k < K; k++) {
       const uint32_t off = (uint32_t)k * G + g;
-      bool chk = trk && off < W && ws + off < n32;
-      if constexpr (GUIDED) chk = chk && ((cb >> k) & 1u);
-      if (chk) {
-        const unsigned long long s0 = __ldcg(S + cr[k]);
-        if ((s0 & ~0xFFFFFFFFull) == tag && (uint32_t)s0 < off) pend |= 1u << k;
-        if constexpr (k2) {
-          const unsigned long long s1 = __ldcg(S + c2[k]);
-          if ((s1 & ~0xFFFFFFFFull) == tag && (uint32_t)s1 < off) pend |= 1u << (K + k);
-        }
-      }
+      if (cur(p0[k], tag) && (uint32_t)p0[k] < off) pend |= 1u << k;
+      if constexpr (k2) if (cur(p1[k], tag) && (uint32_t)p1[k] < off) pend |= 1u << (K + k);
     }
     viol += __popc((pend | (pend >> K)) & ((1u << K) - 1));
+    FTR(3);
     // ---------------- non-violators: values, published where a later reader may wait ----------------
     uint32_t va[K], vt[K];
 #pragma unroll
     for (int k = 0; k < K; k++) {
-      const uint32_t off = (uint32_t)k * G + g;
-      const bool act = off < W && ws + off < n32;
-      if (act && !((pend >> k) & 1u) && !((pend >> (K + k)) & 1u)) {
-        va[k] = fwd_body<OP, DT>(L, g0[k], g1[k], vt[k]);
-        bool pub = trk;
-        if constexpr (GUIDED) pub = pub && ((cb >> (K + k)) & 1u);
-        if (pub) g_st_relaxed(V + cw[k], tag | va[k]);
+      if (act(ws, k) && !(((pend >> k) | (pend >> (K + k))) & 1u)) {
+        va[k] = fwd_body<OP, DT>(L, c.g0[k], c.g1[k], vt[k]);
+        if (trk && src_bit(c, ws, k)) g_st_relaxed(V + c.w[k], tag | va[k]);
       }
     }
+    FTR(4);
     // ---------------- recovery ----------------
+#ifdef JP_TLS_TRACE
+    int npass = 0;
+    const bool anyp = __any_sync(0xffffffffu, pend);
+    FTR(9);
+    if (blockIdx.x == 0 && threadIdx.x == 0 && win < 2048u) g_fwd_trace[win * 16 + 11] = anyp;
+#endif
     while (__any_sync(0xffffffffu, pend)) {
+#ifdef JP_TLS_TRACE
+      npass++;
+#endif
 #pragma unroll
       for (int k = 0; k < K; k++) {
         if (((pend >> k) | (pend >> (K + k))) & 1u) {
           if ((pend >> k) & 1u) {
-            const unsigned long long v = g_ld_relaxed(V + cr[k]);
-            if ((v & ~0xFFFFFFFFull) == tag) { g0[k] = (uint32_t)v; pend &= ~(1u << k); }
+            const unsigned long long v = g_ld_relaxed(V + c.r[k]);
+            if (cur(v, tag)) { c.g0[k] = (uint32_t)v; pend &= ~(1u << k); }
           }
           if constexpr (k2) {
             if ((pend >> (K + k)) & 1u) {
-              const unsigned long long v = g_ld_relaxed(V + c2[k]);
-              if ((v & ~0xFFFFFFFFull) == tag) { g1[k] = (uint32_t)v; pend &= ~(1u << (K + k)); }
+              const unsigned long long v = g_ld_relaxed(V + c.x[k]);
+              if (cur(v, tag)) { c.g1[k] = (uint32_t)v; pend &= ~(1u << (K + k)); }
             }
           }
           if (!(((pend >> k) | (pend >> (K + k))) & 1u)) {
-            va[k] = fwd_body<OP, DT>(L, g0[k], g1[k], vt[k]);
-            bool pub = true;
-            if constexpr (GUIDED) pub = (cb >> (K + k)) & 1u;
-            if (pub) g_st_relaxed(V + cw[k], tag | va[k]);
+            va[k] = fwd_body<OP, DT>(L, c.g0[k], c.g1[k], vt[k]);
+            if (src_bit(c, ws, k)) g_st_relaxed(V + c.w[k], tag | va[k]);
           }
         }
       }
     }
+    FTR(5);
+#ifdef JP_TLS_TRACE
+    if (blockIdx.x == 0 && threadIdx.x == 0 && win < 2048u) g_fwd_trace[win * 16 + 10] = npass;
+#endif
     // ---------------- commit ----------------
 #pragma unroll
     for (int k = 0; k < K; k++) {
-      const uint32_t off = (uint32_t)k * G + g;
-      if (off < W && ws + off < n32) {
-        __stcg(L.A + cw[k], va[k]);
-        if constexpr (OP == JP_OP_PRIV_TMP) __stcg(L.T + c2[k], vt[k]);
+      if (act(ws, k)) {
+        __stcg(L.A + c.w[k], va[k]);
+        if constexpr (OP == JP_OP_PRIV_TMP) __stcg(L.T + c.x[k], vt[k]);
       }
     }
-    // ---------------- forward this window's writes into the next window's operands ----------------
-    uint32_t fx = 0, f0[K], f1[K];
-    if (more && trk) {
+    FTR(6);
+    // ---------------- forward this window's writes into the next window's operands,
+    // then gather the rest of them ----------------
+    uint32_t fwd = 0;
 #pragma unroll
-      for (int k = 0; k < K; k++) {
-        const uint32_t off = (uint32_t)k * G + g;
-        bool chk = off < W && ws + W + off < n32;
-        if constexpr (GUIDED) chk = chk && ((nb >> k) & 1u);
-        if (chk) {
-          if ((__ldcg(S + nr[k]) & ~0xFFFFFFFFull) == tag) {
-            unsigned long long v;
-            do { v = g_ld_relaxed(V + nr[k]); } while ((v & ~0xFFFFFFFFull) != tag);
-            f0[k] = (uint32_t)v;
-            fx |= 1u << k;
-          }
-          if constexpr (k2) {
-            if ((__ldcg(S + n2[k]) & ~0xFFFFFFFFull) == tag) {
-              unsigned long long v;
-              do { v = g_ld_relaxed(V + n2[k]); } while ((v & ~0xFFFFFFFFull) != tag);
-              f1[k] = (uint32_t)v;
-              fx |= 1u << (K + k);
-            }
-          }
+    for (int k = 0; k < K; k++) {
+      if (cur(q0[k], tag)) {
+        unsigned long long v;
+        do { v = g_ld_relaxed(V + nx.r[k]); } while (!cur(v, tag));
+        nx.g0[k] = (uint32_t)v;
+        fwd |= 1u << k;
+      }
+      if constexpr (k2) {
+        if (cur(q1[k], tag)) {
+          unsigned long long v;
+          do { v = g_ld_relaxed(V + nx.x[k]); } while (!cur(v, tag));
+          nx.g1[k] = (uint32_t)v;
+          fwd |= 1u << (K + k);
         }
       }
     }
-#pragma unroll
-    for (int k = 0; k < K; k++) {
-      cr[k] = nr[k]; cw[k] = nw[k];
-      if constexpr (OP == JP_OP_STENCIL2 || OP == JP_OP_PRIV_TMP) c2[k] = n2[k];
-      g0[k] = ((fx >> k) & 1u) ? f0[k] : ng0[k];
-      g1[k] = ((fx >> (K + k)) & 1u) ? f1[k] : ng1[k];
-    }
-    cb = nb;
-    if (win + 2 < nwin) load_idx(ws + 2 * W, nr, nw, n2, nb);
+    if (more) gather(ws + W, nx, fwd);
+    FTR(7);
+    if (win + 2 < nwin) load_idx(ws + 2 * W, c);
+    FTR(8);
+  }
+};
+
+template <int OP, int DT, bool GUIDED>
+__global__ void __launch_bounds__(kFwdThreads, 1)
+    k_tls_fwd_grid(DLoop L, int track, uint32_t W, const uint32_t *graw, const uint32_t *gsrc, unsigned long long *S,
+                   unsigned long long *V, unsigned *bar, int64_t *stats) {
+  constexpr int K = kFwdK;
+  FwdGrid<OP, DT, GUIDED, K> F;
+  F.L = L; F.graw = graw; F.gsrc = gsrc; F.S = S; F.V = V; F.bar = bar;
+  F.W = W;
+  F.G = gridDim.x * (uint32_t)kFwdThreads;
+  F.g = blockIdx.x * (uint32_t)kFwdThreads + threadIdx.x;
+  F.n32 = (uint32_t)L.n;
+  F.io = (uint32_t)L.ioff;
+  F.nwin = (F.n32 + W - 1) / W;
+  F.trk = FwdGrid<OP, DT, GUIDED, K>::kTr && track;
+  FwdSet<K> A, B;
+  F.load_idx(0, A);
+  F.gather(0, A);
+  if (F.nwin > 1) F.load_idx(W, B);
+  for (uint32_t win = 0; win < F.nwin; win += 2) {
+    F.step(win, A, B);
+    if (win + 1 < F.nwin) F.step(win + 1, B, A);
   }
   // ---------------- stats: stats[3] and the dup counter (bar[1]) were zeroed by the launcher ----------------
-  viol = __reduce_add_sync(0xffffffffu, viol);
-  dup = __reduce_add_sync(0xffffffffu, dup);
+  const int tid = threadIdx.x;
+  uint32_t viol = __reduce_add_sync(0xffffffffu, F.viol);
+  uint32_t dup = __reduce_add_sync(0xffffffffu, F.dup);
   if ((tid & 31) == 0) {
     if (viol) atomicAdd(reinterpret_cast<unsigned long long *>(&stats[3]), (unsigned long long)viol);
     if (dup) atomicAdd(bar + 1, dup);
   }
-  fwd_grid_sync(bar, gridDim.x * (nwin + 1));
+  fwd_grid_sync(bar, gridDim.x * (F.nwin + 1));
   if (blockIdx.x == 0 && tid == 0) {
     const int64_t v = *(volatile int64_t *)&stats[3];
-    stats[0] = *(volatile unsigned *)(bar + 1) ? -1 : (int64_t)n32;
-    stats[1] = (int64_t)n32 + v;
-    stats[2] = nwin;
+    stats[0] = *(volatile unsigned *)(bar + 1) ? -1 : (int64_t)F.n32;
+    stats[1] = (int64_t)F.n32 + v;
+    stats[2] = F.nwin;
   }
 }
 

@@ -68,3 +68,20 @@ def main():
 
 if __name__ == "__main__":
     main()
+
+
+def doall_floor():
+    """The same body and index shape with no dependence (config 3 at d = 0) run as
+    DOALL: the random gather + scatter floor the TLS path is measured against."""
+    dev = torch.device("cuda:0")
+    st = torch.cuda.current_stream()
+    wl = synth.config3(0.0, device=dev)
+    L = jp.Loop.from_workload(wl)
+    ws = jp.workspace(L)
+    prof = jp.jp_profile_density(L, ws)
+    ms, _ = ev_ms(lambda pre: None if pre else jp.jp_run_doall(L, prof, ws, stream=st), st, reps=5)
+    print(json.dumps({"doall_indirect_d0": {"ms": round(ms, 3), "Giter_s": round(wl.n / ms / 1e6, 2)}}), flush=True)
+
+
+if __name__ == "__main__" and os.environ.get("DOALL_FLOOR"):
+    doall_floor()
