@@ -17,13 +17,29 @@
 // with two steps in flight and 32-bit index arithmetic.
 // The intra-warp / inter-warp split of the paper is an
 // implementation detail here (reading A2): results do not depend on geometry.
+#include <cstdlib>
 #include "jp_host.h"
 
 namespace jp {
 
+// table bytes stamped per pass (env JP_STAMP_PASS_MB overrides, for measurement)
+static size_t stamp_pass_bytes() {
+  static size_t v = [] {
+    const char *e = getenv("JP_STAMP_PASS_MB");
+    const long mb = e ? atol(e) : 48;
+    return (size_t)(mb > 0 ? mb : 48) << 20;
+  }();
+  return v;
+}
+
 struct Tabs {
   int32_t *wA, *rA, *wT, *rT;
   int sA, sT;   // pre-aggregate in shared memory
+  // stamp pass over an address window [lo, lo + span) only (tables larger than
+  // L2 are stamped in several passes, each with an L2-resident working set);
+  // index errors are counted by the pass with count_bad
+  uint32_t lo, span;
+  int count_bad;
 };
 
 __device__ __forceinline__ void check(int64_t a, int64_t len, int64_t &bad) {
@@ -55,9 +71,10 @@ __device__ __forceinline__ int4 idx4(const DLoop &L, const int32_t *p, int64_t i
 }
 __device__ __forceinline__ int q4(const int4 &v, int k) { return k == 0 ? v.x : k == 1 ? v.y : k == 2 ? v.z : v.w; }
 // chk: the index came from an index array (identity indices were range-checked on the host)
-__device__ __forceinline__ void stamp32(int32_t *g, int32_t *s, int32_t a, int32_t len, int32_t e, int &bad,
-                                        bool chk = true) {
-  if (chk && (uint32_t)a >= (uint32_t)len) { bad++; return; }
+__device__ __forceinline__ void stamp32(int32_t *g, int32_t *s, int32_t a, int32_t len, int32_t e, const Tabs &t,
+                                        int &bad, bool chk = true) {
+  if (chk && (uint32_t)a >= (uint32_t)len) { bad += t.count_bad; return; }
+  if ((uint32_t)a - t.lo >= t.span) return;
   if (s) {
     if (s[a] < e) atomicMax(&s[a], e);
   } else if (g) {
@@ -109,29 +126,29 @@ __global__ void __launch_bounds__(256) k_prof_stamp4(DLoop L, Tabs t, int vec, i
         // identity streams (NULL arrays) were range-checked on the host and
         // reach a table only when the array is also reached through an index
         if constexpr (OP == JP_OP_ADD_C) {
-          stamp32(t.wA, sAw, a, lenA, e, bad, hw);
-          stamp32(t.rA, sAr, b, lenA, e, bad, hr);
+          stamp32(t.wA, sAw, a, lenA, e, t, bad, hw);
+          stamp32(t.rA, sAr, b, lenA, e, t, bad, hr);
         } else if constexpr (OP == JP_OP_SAXPY) {
           if (hr && (uint32_t)b >= (uint32_t)lenX) bad++;
           if (hw) {
-            stamp32(t.wA, sAw, a, lenA, e, bad);
-            if ((uint32_t)a < (uint32_t)lenA) stamp32(t.rA, sAr, a, lenA, e, bad, false);
+            stamp32(t.wA, sAw, a, lenA, e, t, bad);
+            if ((uint32_t)a < (uint32_t)lenA) stamp32(t.rA, sAr, a, lenA, e, t, bad, false);
           }
         } else if constexpr (OP == JP_OP_PRIV_TMP) {
           if (hr && (uint32_t)b >= (uint32_t)lenX) bad++;
           if (h2) {
             if (sTw) {
-              stamp32(t.wT, sTw, a, lenT, e, bad);
+              stamp32(t.wT, sTw, a, lenT, e, t, bad);
             } else {
-              stamp32(t.wT, nullptr, a, lenT, e, bad);
-              if ((uint32_t)a < (uint32_t)lenT) stamp32(t.rT, nullptr, a, lenT, e, bad, false);
+              stamp32(t.wT, nullptr, a, lenT, e, t, bad);
+              if ((uint32_t)a < (uint32_t)lenT) stamp32(t.rT, nullptr, a, lenT, e, t, bad, false);
             }
           }
-          if (hw) stamp32(t.wA, sAw, q4(vc[u], k), lenA, e, bad);
+          if (hw) stamp32(t.wA, sAw, q4(vc[u], k), lenA, e, t, bad);
         } else {
-          stamp32(t.wA, sAw, a, lenA, e, bad, hw);
-          stamp32(t.rA, sAr, b, lenA, e, bad, hr);
-          stamp32(t.rA, sAr, q4(vc[u], k), lenA, e, bad, h2);
+          stamp32(t.wA, sAw, a, lenA, e, t, bad, hw);
+          stamp32(t.rA, sAr, b, lenA, e, t, bad, hr);
+          stamp32(t.rA, sAr, q4(vc[u], k), lenA, e, t, bad, h2);
         }
       }
     }
@@ -449,6 +466,9 @@ static void run_stamp(const DLoop &d, Tabs t, int64_t *hdr, size_t smem, cudaStr
 
 static Tabs tabs_of(const DLoop &d, void *ws, const Layout &lo) {
   Tabs t;
+  t.lo = 0;
+  t.span = 0xFFFFFFFFu;
+  t.count_bad = 1;
   t.wA = at<int32_t>(ws, lo, R_MINW_A);
   t.rA = at<int32_t>(ws, lo, R_MINR_A);
   t.wT = at<int32_t>(ws, lo, R_MINW_T);
@@ -462,14 +482,29 @@ cudaError_t launch_prof_stamp(const Job &j, void *ws, const Layout &lo, cudaStre
   int64_t *hdr = at<int64_t>(ws, lo, R_HEADER);
   cudaMemsetAsync(hdr, 0, kHeaderBytes, st);
   cudaMemsetAsync(&hdr[H_FIRST_RAW], 0xFF, sizeof(int64_t), st);   // none (= ~0 for the u64 atomicMin)
-  for (int r = R_MINW_A; r <= R_MINR_T; r++)
+  size_t tab_bytes = 0;
+  for (int r = R_MINW_A; r <= R_MINR_T; r++) {
     if (lo.bytes[r]) cudaMemsetAsync(static_cast<char *>(ws) + lo.off[r], 0xFF, lo.bytes[r], st);
+    tab_bytes += lo.bytes[r];
+  }
   if (j.d.n == 0) return launch_check();
   Tabs t = tabs_of(j.d, ws, lo);
   size_t smem = 0;
   if (t.sA) smem += (size_t)j.d.lenA * 4 * (t.rA ? 2 : 1);
   if (t.sT) smem += (size_t)j.d.lenT * 4;
-  JP_DISPATCH(j.op, j.dt, run_stamp, j.d, t, hdr, smem, st);
+  // tables beyond ~48 MB (a third of L2) are stamped one address window at a
+  // time: every pass re-streams the index arrays but its random atomics hit L2
+  const int64_t amax = std::max(j.d.lenA, j.d.lenT);
+  const size_t pb = stamp_pass_bytes();
+  int np = (t.sA || t.sT) ? 1 : (int)((tab_bytes + pb - 1) / pb);
+  if (np < 1) np = 1;
+  const int64_t step = (amax + np - 1) / np;
+  for (int p = 0; p < np; p++) {
+    t.lo = (uint32_t)(p * step);
+    t.span = np == 1 ? 0xFFFFFFFFu : (uint32_t)step;
+    t.count_bad = p == 0;
+    JP_DISPATCH(j.op, j.dt, run_stamp, j.d, t, hdr, smem, st);
+  }
   return launch_check();
 }
 
