@@ -757,9 +757,14 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
   char *sch = static_cast<char *>(ws) + lo.off[R_SCHED];
   const int64_t nck = (L->n + chunk - 1) / chunk;
   int64_t *cc = reinterpret_cast<int64_t *>(sch + sl.counts);
-  // 1. profile with per-chunk counts (global stamps, reading A19)
+  // 1. profile with per-chunk counts (global stamps, reading A19); the classify
+  //    pass also writes the TLS guide bitmaps when the loop can be guided
+  const bool gfuse = lo.bytes[R_GUIDE] && c.tls_recovery != 1 && j.op != JP_OP_PRIV_TMP &&
+                     a_indirect(j.op, j.d.r, j.d.r2, j.d.w);
+  uint32_t *gbits = gfuse ? at<uint32_t>(ws, lo, R_GUIDE) : nullptr;
   JP_CUDA(launch_prof_stamp(j, ws, lo, st), "profile stamp");
-  JP_CUDA(launch_prof_classify(j, ws, lo, nullptr, chunk, cc, st), "profile classify");
+  JP_CUDA(launch_prof_classify(j, ws, lo, gbits, chunk, cc, st, gbits ? gbits + (L->n + 31) / 32 : nullptr),
+          "profile classify");
   std::vector<int64_t> hc(3 * nck), h(8);
   JP_CUDA(cudaMemcpyAsync(hc.data(), cc, 24 * nck, cudaMemcpyDeviceToHost, st), "chunk D2H");
   JP_CUDA(cudaMemcpyAsync(h.data(), at<int64_t>(ws, lo, R_HEADER), 64, cudaMemcpyDeviceToHost, st), "profile D2H");
@@ -801,7 +806,8 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
     JP_CUDA(cudaMemcpyAsync(dct, ct.data(), 4 * nck, cudaMemcpyHostToDevice, st), "task map H2D");
     auto P = [&](size_t o) { return o == SIZE_MAX ? nullptr : reinterpret_cast<unsigned long long *>(sch + o); };
     unsigned long long *dconf = P(sl.conf);
-    JP_CUDA(launch_task_conflicts(j, dct, chunk, P(sl.wmA), P(sl.rmA), P(sl.wmT), P(sl.rmT), dconf, st), "conflicts");
+    JP_CUDA(launch_task_conflicts(j, dct, chunk, nt, P(sl.wmA), P(sl.rmA), P(sl.wmT), P(sl.rmT), dconf, st),
+            "conflicts");
     JP_CUDA(cudaMemcpyAsync(conf.data(), dconf, 8 * kMaxTasks, cudaMemcpyDeviceToHost, st), "conf D2H");
     JP_CUDA(cudaStreamSynchronize(st), "conf sync");
   }
@@ -816,12 +822,11 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
   // 4. run batch by batch; tasks of one batch are pairwise conflict-free and run
   //    concurrently (TLS on one SM, partitioned modes on the rest)
   int64_t *tstats = reinterpret_cast<int64_t *>(sch + sl.tstats);
-  // guide bitmaps for on-chip TLS tasks (from this profile's stamp tables)
-  bool guided_ok = false;
-  for (int t = 0; t < nt && !guided_ok; t++) guided_ok = tasks[t].mode == JP_MODE_TLS;
-  guided_ok = guided_ok && c.tls_recovery != 1 && lo.bytes[R_GUIDE] && j.op != JP_OP_PRIV_TMP &&
-              a_indirect(j.op, j.d.r, j.d.r2, j.d.w);
-  if (guided_ok) JP_CUDA(launch_tls_guide(j, ws, lo, st), "tls guide");
+  // on-chip TLS tasks use the guide bitmaps of step 1 (valid for them: no
+  // iteration of such a task writes an address written earlier in the loop, so
+  // its writers of raw-read addresses are first writers)
+  const bool guided_ok = gfuse;
+  std::vector<int> grid_tls;   // on-chip TLS tasks, run on every SM after the batch's other tasks
   cudaEvent_t ev0;
   JP_CUDA(cudaEventCreateWithFlags(&ev0, cudaEventDisableTiming), "event");
   std::vector<cudaEvent_t> evs;
@@ -853,20 +858,11 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
           for (int64_t k = tasks[t].s / chunk; k * chunk < tasks[t].e; k++) { tprof.raw_iters += hc[3 * k]; tprof.waw_iters += hc[3 * k + 2]; }
           const bool onchip = c.tls_recovery == 2 || (c.tls_recovery == 0 && c.tls_path == 0 && tprof.waw_iters == 0);
           if (onchip) {
-            // on-chip recovery (reading B7) on one cluster beside the partitioned tasks, guided by
-            // the whole loop's bitmaps (the task starts on a chunk boundary, a multiple of 32)
-            jp_tls_cfg tc{c.tls_window, 0, 5, 0, 0, JP_TLS_ONCHIP};
-            JP_TRY(tls_plan(sj, &tc, &tprof, tp));
-            const uint32_t *gb = guided_ok ? at<uint32_t>(ws, lo, R_GUIDE) : nullptr;
-            const int64_t nw = (L->n + 31) / 32;
-            res->tls_w_max = tp.window;
-            res->tls_path = 5;
-            res->tls_recovery = JP_TLS_ONCHIP;
-            res->tls_cluster = tp.cluster;
-            res->tls_guided = gb ? 1 : 0;
-            JP_CUDA(launch_tls_fwd(sj, tp.window, tp.cluster, gb ? gb + tasks[t].s / 32 : nullptr,
-                                   gb ? gb + nw + tasks[t].s / 32 : nullptr, tstats + 4 * t, s2),
-                    "tls task");
+            // on-chip recovery (reading B7) uses every SM: it runs after the
+            // batch's partitioned tasks (below), on the caller's stream
+            grid_tls.push_back(t);
+            res->task_mode_iters[tasks[t].mode] += sj.d.n;
+            continue;
           } else {
             // the single-CTA path (one SM, beside the partitioned tasks), window cap from the task's density
             const int64_t wm = c.tls_w_max > 0 ? c.tls_w_max : auto_w_max(tprof.raw_iters >= 0 ? &tprof : nullptr);
@@ -891,6 +887,34 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
       }
     }
     for (auto e : joins) cudaStreamWaitEvent(st, e, 0);
+    for (int t : grid_tls) {
+      if (level[t] != lv) continue;
+      // guided by the whole loop's bitmaps (the task starts on a chunk boundary, a multiple of 32)
+      Job sj = sub_job(j, tasks[t].s, tasks[t].e);
+      TlsPlan tp;
+      jp_profile tprof{};
+      tprof.n = sj.d.n;
+      jp_tls_cfg tc{c.tls_window, 0, 0, 0, 0, JP_TLS_ONCHIP};
+      JP_TRY(tls_plan(sj, &tc, &tprof, tp));
+      const uint32_t *gb = guided_ok ? at<uint32_t>(ws, lo, R_GUIDE) : nullptr;
+      const int64_t nw = (L->n + 31) / 32;
+      const uint32_t *b0 = gb ? gb + tasks[t].s / 32 : nullptr, *b1 = gb ? gb + nw + tasks[t].s / 32 : nullptr;
+      if (tp.path == 6) {
+        JP_CUDA(launch_tls_fwd_grid(sj, tp.window, b0, b1, at<unsigned long long>(ws, lo, R_TLS_S_A),
+                                    at<unsigned long long>(ws, lo, R_TLS_C_A), L->len_A,
+                                    reinterpret_cast<unsigned *>(&at<int64_t>(ws, lo, R_HEADER)[H_BAR_COUNT]),
+                                    tstats + 4 * t, st),
+                "tls task");
+      } else {
+        JP_CUDA(launch_tls_fwd(sj, tp.window, tp.cluster, b0, b1, tstats + 4 * t, st), "tls task");
+      }
+      res->tls_w_max = tp.window;
+      res->tls_path = tp.path;
+      res->tls_recovery = JP_TLS_ONCHIP;
+      res->tls_cluster = tp.cluster;
+      res->tls_guided = gb ? 1 : 0;
+      tls_tasks.push_back(t);
+    }
     if (any_priv) JP_CUDA(launch_priv_finalize(j, ws, lo, st), "priv finalize");
   }
   // stats of the TLS tasks

@@ -48,8 +48,9 @@ cudaError_t launch_validate(const Job &j, int64_t *hdr, cudaStream_t st);
 // stamp tables of a profile on the same workspace; no sync.
 cudaError_t launch_tls_guide(const Job &j, void *ws, const Layout &lo, cudaStream_t st);
 cudaError_t launch_prof_stamp(const Job &j, void *ws, const Layout &lo, cudaStream_t st);
+// src_bits (nullable): also the TLS guide's RAW-source words (raw_bits then holds its raw words)
 cudaError_t launch_prof_classify(const Job &j, void *ws, const Layout &lo, uint32_t *raw_bits,
-                                 int64_t chunk, int64_t *chunk_counts, cudaStream_t st);
+                                 int64_t chunk, int64_t *chunk_counts, cudaStream_t st, uint32_t *src_bits = nullptr);
 // counts + the TLS guide bitmaps (region 13, valid when the loop writes no address twice) in one pass
 cudaError_t launch_prof_classify_guide(const Job &j, void *ws, const Layout &lo, cudaStream_t st);
 cudaError_t launch_doall(const Job &j, cudaStream_t st, int max_ctas = 0);
@@ -64,7 +65,7 @@ cudaError_t launch_merge_apply(void *arr, int64_t len, const int64_t *keys, cuda
 // STEALING scheduler helpers (jp_sched.cu): per-task write/read bitmasks of every
 // address, then the task x task conflict matrix conf[t] (bit u set: t and u
 // touch a common address and at least one of them writes it).
-cudaError_t launch_task_conflicts(const Job &j, const int32_t *chunk_task, int64_t chunk,
+cudaError_t launch_task_conflicts(const Job &j, const int32_t *chunk_task, int64_t chunk, int n_tasks,
                                   unsigned long long *wmA, unsigned long long *rmA,
                                   unsigned long long *wmT, unsigned long long *rmT,
                                   unsigned long long *conf, cudaStream_t st);

@@ -286,9 +286,11 @@ __device__ __forceinline__ bool earlier(const int32_t *tab, int64_t a, int64_t l
   return tab && (uint64_t)a < (uint64_t)len && tab[a] > e;
 }
 
+// src_bits (nullable, zeroed by the caller): the RAW-source words of the TLS
+// guide, OR-ed in at the first writer of every raw read (see k_prof_count4)
 template <int OP>
 __global__ void __launch_bounds__(256) k_prof_classify(DLoop L, Tabs t, uint32_t *raw_bits, int64_t chunk,
-                                                        int64_t *chunk_counts, int64_t *hdr) {
+                                                        int64_t *chunk_counts, int64_t *hdr, uint32_t *src_bits) {
   __shared__ unsigned long long s_cnt[3];
   __shared__ unsigned long long s_first;
   if (threadIdx.x < 3) s_cnt[threadIdx.x] = 0;
@@ -321,21 +323,32 @@ __global__ void __launch_bounds__(256) k_prof_classify(DLoop L, Tabs t, uint32_t
       raw[u] = war[u] = waw[u] = false;
       if (i < L.n) {
         const int32_t e = enc_gid(L.base + i);
+        auto src = [&](int64_t a) {   // mark the first writer of a raw read's address
+          if (src_bits) {
+            const int64_t jw = (int64_t)(0x7FFFFFFF - t.wA[a]) - L.base;
+            atomicOr(&src_bits[jw >> 5], 1u << (jw & 31));
+          }
+        };
         if constexpr (OP == JP_OP_ADD_C) {
           raw[u] = earlier(t.wA, ib[u], L.lenA, e);
           war[u] = earlier(t.rA, ia[u], L.lenA, e);
           waw[u] = earlier(t.wA, ia[u], L.lenA, e);
+          if (raw[u]) src(ib[u]);
         } else if constexpr (OP == JP_OP_SAXPY) {
           raw[u] = earlier(t.wA, ia[u], L.lenA, e);
           war[u] = earlier(t.rA, ia[u], L.lenA, e);
           waw[u] = raw[u];   // the same address is the exposed read and the write
+          if (raw[u]) src(ia[u]);
         } else if constexpr (OP == JP_OP_PRIV_TMP) {
           war[u] = earlier(rT, ia[u], L.lenT, e);
           waw[u] = earlier(t.wT, ia[u], L.lenT, e) || earlier(t.wA, ib[u], L.lenA, e);
         } else {
-          raw[u] = earlier(t.wA, ib[u], L.lenA, e) || earlier(t.wA, ic[u], L.lenA, e);
+          const bool r0 = earlier(t.wA, ib[u], L.lenA, e), r1 = earlier(t.wA, ic[u], L.lenA, e);
+          raw[u] = r0 || r1;
           war[u] = earlier(t.rA, ia[u], L.lenA, e);
           waw[u] = earlier(t.wA, ia[u], L.lenA, e);
+          if (r0) src(ib[u]);
+          if (r1) src(ic[u]);
         }
       }
     }
@@ -510,7 +523,7 @@ cudaError_t launch_prof_stamp(const Job &j, void *ws, const Layout &lo, cudaStre
 
 template <int OP, int DT>
 static void run_classify(const DLoop &d, Tabs t, uint32_t *bits, int64_t chunk, int64_t *cc, int64_t *hdr,
-                         cudaStream_t st) {
+                         uint32_t *src_bits, cudaStream_t st) {
   (void)DT;
   int64_t tiles = (d.n + 31) / 32;
   if (!bits && !cc) {
@@ -518,20 +531,22 @@ static void run_classify(const DLoop &d, Tabs t, uint32_t *bits, int64_t chunk, 
     k_prof_count4<OP, false><<<grid_for((nq + kQuadSteps - 1) / kQuadSteps, 256, 8), 256, 0, st>>>(d, t, idx_vec(d), hdr,
                                                                                                  nullptr, nullptr);
   } else {
-    k_prof_classify<OP><<<grid_for((tiles + kUnroll - 1) / kUnroll * 32, 256, 8), 256, 0, st>>>(d, t, bits, chunk, cc, hdr);
+    k_prof_classify<OP><<<grid_for((tiles + kUnroll - 1) / kUnroll * 32, 256, 8), 256, 0, st>>>(d, t, bits, chunk, cc, hdr,
+                                                                                                 src_bits);
   }
   note_launch();
 }
 
 cudaError_t launch_prof_classify(const Job &j, void *ws, const Layout &lo, uint32_t *raw_bits, int64_t chunk,
-                                 int64_t *chunk_counts, cudaStream_t st) {
+                                 int64_t *chunk_counts, cudaStream_t st, uint32_t *src_bits) {
   int64_t *hdr = at<int64_t>(ws, lo, R_HEADER);
   cudaMemsetAsync(&hdr[H_RAW], 0, 3 * sizeof(int64_t), st);
   cudaMemsetAsync(&hdr[H_FIRST_RAW], 0xFF, sizeof(int64_t), st);
   if (chunk_counts) cudaMemsetAsync(chunk_counts, 0, sizeof(int64_t) * 3 * ((j.d.n + chunk - 1) / chunk), st);
   if (j.d.n == 0) return launch_check();
   Tabs t = tabs_of(j.d, ws, lo);
-  JP_DISPATCH(j.op, j.dt, run_classify, j.d, t, raw_bits, chunk, chunk_counts, hdr, st);
+  if (src_bits) cudaMemsetAsync(src_bits, 0, 4 * (size_t)((j.d.n + 31) / 32), st);
+  JP_DISPATCH(j.op, j.dt, run_classify, j.d, t, raw_bits, chunk, chunk_counts, hdr, src_bits, st);
   return launch_check();
 }
 

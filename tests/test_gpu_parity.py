@@ -565,7 +565,7 @@ def test_schedule_stealing_config5(n, chunk, recovery):
     b, e = n // 2, 3 * n // 4   # the TLS task, as a loop of its own
     mid = O.Loop(ref.op, ref.dtype, e - b, ref.A, r=ref.r[b:e], w=ref.w[b:e], c0=ref.c0)
     if recovery == 0:
-        assert res["tls_recovery"] == jp.JP_TLS_ONCHIP and res["tls_path"] == 5 and res["tls_guided"] == 1
+        assert res["tls_recovery"] == jp.JP_TLS_ONCHIP and res["tls_path"] in (5, 6) and res["tls_guided"] == 1
         assert res["tls"] == O.sim_tls_fwd(mid, res["tls_w_max"])[3]
     else:
         assert res["tls_recovery"] == jp.JP_TLS_RESTART and res["tls_path"] == 1
@@ -724,3 +724,35 @@ def test_tiny_recovery_and_windows(kw):
     if kw.get("tls_window"):
         assert res["tls"]["windows"] >= -(-4096 // kw["tls_window"])
     tiny_case(random_loop(41, O.OP_STENCIL2, O.F32, 3000, len_a=6000, null_prob=0.0, dup_writes=False), **kw)
+
+
+@pytest.mark.parametrize("cross", [False, True])
+def test_schedule_stealing_many_tasks(cross):
+    """32 alternating DOALL / TLS chunk tasks (64-bit task masks; <= 8 tasks use
+    byte masks): disjoint address blocks give one batch; with `cross`, each TLS
+    chunk also reads what the previous DOALL chunk wrote, ordering the tasks."""
+    n, chunk = 32768, 1024
+    g = np.random.default_rng(9)
+    r = np.empty(n, np.int32)
+    w = np.empty(n, np.int32)
+    for c in range(n // chunk):
+        base = c * chunk
+        if c % 2 == 0:   # DOALL: a permutation of the block, read = write address
+            p = g.permutation(chunk).astype(np.int32) + base
+            r[base:base + chunk] = p
+            w[base:base + chunk] = p
+        else:            # TLS: a prefix chain inside the block
+            w[base:base + chunk] = np.arange(base, base + chunk, dtype=np.int32)
+            r[base:base + chunk] = np.maximum(np.arange(base - 1, base + chunk - 1, dtype=np.int32), base)
+            if cross:
+                r[base] = base - chunk + 5   # the previous (DOALL) block's write
+    wl = synth.Workload("alt", O.OP_ADD_C, O.I32, n, torch.arange(n, dtype=torch.int32) * 5,
+                        r=torch.from_numpy(r), w=torch.from_numpy(w), c0=3)
+    _, A, T = O.run_seq(to_oracle(wl))
+    gw = gpu(wl)
+    L = jp.Loop.from_workload(gw)
+    res = jp.jp_schedule(L, jp.workspace(L), scheme=jp.JP_SCHED_STEALING, chunk_iters=chunk)
+    torch.cuda.synchronize()
+    check_arrays(gw, A, T)
+    assert res["n_tasks"] == n // chunk
+    assert res["n_batches"] == (2 if cross else 1)
