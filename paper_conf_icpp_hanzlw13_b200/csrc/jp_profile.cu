@@ -24,12 +24,9 @@ namespace jp {
 
 // table bytes stamped per pass (env JP_STAMP_PASS_MB overrides, for measurement)
 static size_t stamp_pass_bytes() {
-  static size_t v = [] {
-    const char *e = getenv("JP_STAMP_PASS_MB");
-    const long mb = e ? atol(e) : 48;
-    return (size_t)(mb > 0 ? mb : 48) << 20;
-  }();
-  return v;
+  const char *e = getenv("JP_STAMP_PASS_MB");
+  const long mb = e ? atol(e) : 48;
+  return (size_t)(mb > 0 ? mb : 48) << 20;
 }
 
 struct Tabs {

@@ -756,3 +756,38 @@ def test_schedule_stealing_many_tasks(cross):
     check_arrays(gw, A, T)
     assert res["n_tasks"] == n // chunk
     assert res["n_batches"] == (2 if cross else 1)
+
+
+@pytest.mark.parametrize("pass_mb", ["1", "3"])
+def test_profile_address_windows(pass_mb, monkeypatch):
+    """The stamp pass in L2-sized address windows (forced small with
+    JP_STAMP_PASS_MB): counts and the first raw iteration equal the oracle's;
+    a whole jp_schedule (fused guide bitmaps, on-chip TLS) stays exact."""
+    monkeypatch.setenv("JP_STAMP_PASS_MB", pass_mb)
+    for wl in (synth.config3(0.05, n=(1 << 19) + 5), synth.config5(n=1 << 19),
+               random_loop(61, O.OP_STENCIL2, O.F32, 300000, len_a=1 << 19, null_prob=0.0),
+               random_loop(62, O.OP_SAXPY, O.I32, 300000, len_a=1 << 19, null_prob=0.0)):
+        ref = to_oracle(wl)
+        pr = O.profile(ref)
+        g = gpu(wl)
+        L = jp.Loop.from_workload(g)
+        ws = jp.workspace(L)
+        p = jp.jp_profile_density(L, ws)
+        assert (p["raw_iters"], p["war_iters"], p["waw_iters"], p["first_raw_iter"]) == \
+            (pr["raw_iters"], pr["war_iters"], pr["waw_iters"], pr["first_raw_iter"])
+        _, A, T = O.run_seq(ref)
+        res = jp.jp_schedule(L, ws)
+        torch.cuda.synchronize()
+        check_arrays(g, A, T)
+        assert res["prof"]["raw_iters"] == pr["raw_iters"]
+
+
+def test_profile_config3_full_size():
+    """BASELINE size (N = 2^24, tables 2 x 64 MiB: the windowed passes) against the oracle."""
+    wl = synth.config3(0.05)
+    pr = O.profile(to_oracle(wl))
+    g = gpu(wl)
+    L = jp.Loop.from_workload(g)
+    p = jp.jp_profile_density(L, jp.workspace(L))
+    assert (p["raw_iters"], p["war_iters"], p["waw_iters"], p["first_raw_iter"]) == \
+        (pr["raw_iters"], pr["war_iters"], pr["waw_iters"], pr["first_raw_iter"])
