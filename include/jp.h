@@ -139,7 +139,9 @@ typedef struct {
   int32_t tls_recovery;         /* 0 auto (JP_TLS_ONCHIP when the profile shows
                                    waw_iters == 0, else JP_TLS_RESTART), 1 restart,
                                    2 on-chip                                      */
-  int32_t reserved;
+  int32_t static_check;         /* 0: jp_static_check before profiling (affine,
+                                   conflict-free loops run as DOALL unprofiled);
+                                   1: skip it                                     */
 } jp_sched_cfg;
 
 typedef struct {
@@ -213,6 +215,29 @@ jp_status jp_profile_density(const jp_loop *L, void *ws, size_t ws_bytes, uint32
  * (D').  p may be NULL only for the all-NULL case (else JP_ERR_ARG -> -1).   */
 int32_t jp_select_mode(const jp_loop *L /* host */, const jp_profile *p /* host, nullable */,
                        double tau_high);
+
+/* ---- static analysis lite (P:L253-256 rule 1, mode A
+ * "determined DOALL by static analysis" P:L360-362) -----------------------------
+ * One streaming pass decides whether every non-NULL index array is affine in
+ * the loop variable (p[i] == alpha*i + beta for all i); NULL arrays are the
+ * identity (alpha 1, beta ident_off).  When all are, an exact integer test of
+ * every (write, access) pair of the same array (a solution i != j in [0, n) of
+ * alpha_f*i + beta_f == alpha_g*j + beta_g) decides `independent`; `in_range`
+ * checks every affine index against its array from the endpoints.  syncs.
+ * jp_schedule runs it before profiling (jp_sched_cfg.static_check == 0) and
+ * executes an independent, in-range loop as DOALL without a profile.       */
+typedef struct {
+  int32_t affine;               /* 1: every index array is affine                    */
+  int32_t independent;          /* 1: affine and free of cross-iteration conflicts   */
+  int32_t in_range;             /* 1: affine and every index inside its array        */
+  int32_t reserved;
+  int64_t alpha[4], beta[4];    /* r, r2, w, s (meaningful when affine)              */
+} jp_static;
+jp_status jp_static_check(const jp_loop *L, void *ws, size_t ws_bytes, jp_static *out /* host */,
+                          jp_stream_t st);
+/* The exact test it uses (host only, no device): 1 iff some i != j in [0, n)
+ * has af*i + bf == ag*j + bg (|alpha|, |beta| < 2^31, n < 2^31).              */
+int32_t jp_affine_dependence(int64_t af, int64_t bf, int64_t ag, int64_t bg, int64_t n);
 
 /* ---- DOALL -------------------------------------------------------
  * Executes all n iterations in place with no protection.  With a profile (host,

@@ -173,6 +173,20 @@ def jp_select_mode(loop: Loop, prof=None, tau_high: float = 0.25) -> int:
     return m
 
 
+def jp_static_check(loop: Loop, ws, stream=None) -> dict:
+    """Static analysis lite (jp.h): affine index arrays and an exact dependence test."""
+    out = _abi.jp_static()
+    p, nb = _ws(ws)
+    check(lib().jp_static_check(loop.ref, p, nb, C.byref(out), _stream(stream)))
+    return {"affine": out.affine, "independent": out.independent, "in_range": out.in_range,
+            "alpha": list(out.alpha), "beta": list(out.beta)}
+
+
+def jp_affine_dependence(af: int, bf: int, ag: int, bg: int, n: int) -> bool:
+    """Host-only exact test: some i != j in [0, n) with af*i + bf == ag*j + bg."""
+    return bool(lib().jp_affine_dependence(int(af), int(bf), int(ag), int(bg), int(n)))
+
+
 def jp_run_doall(loop: Loop, prof=None, ws=None, stream=None):
     p, nb = _ws(ws)
     check(lib().jp_run_doall(loop.ref, _pref(prof), p, nb, _stream(stream)))
@@ -229,10 +243,11 @@ def jp_run_tls(loop: Loop, window=0, w_max=65536, path=0, prof=None, ws=None, st
 
 
 def sched_cfg(scheme=JP_SCHED_SHARING, tau_high=0.25, chunk_iters=65536, tls_window=0, tls_w_max=0,
-              tls_path=0, tls_recovery=0) -> _abi.jp_sched_cfg:
-    """tls_recovery: 0 auto (on chip when the profile shows waw_iters == 0), 1 restart, 2 on chip."""
+              tls_path=0, tls_recovery=0, static_check=0) -> _abi.jp_sched_cfg:
+    """tls_recovery: 0 auto (on chip when the profile shows waw_iters == 0), 1 restart, 2 on chip.
+    static_check: 0 run jp_static_check before profiling, 1 skip it."""
     return _abi.jp_sched_cfg(int(scheme), int(tls_path), float(tau_high), int(chunk_iters), int(tls_window),
-                             int(tls_w_max), int(tls_recovery), 0)
+                             int(tls_w_max), int(tls_recovery), int(static_check))
 
 
 def _res_dict(r: _abi.jp_sched_result) -> dict:

@@ -63,7 +63,12 @@ class jp_tls_cfg(C.Structure):
 class jp_sched_cfg(C.Structure):
     _fields_ = [("scheme", C.c_int32), ("tls_path", C.c_int32), ("tau_high", C.c_double),
                 ("chunk_iters", C.c_int64), ("tls_window", C.c_int64), ("tls_w_max", C.c_int64),
-                ("tls_recovery", C.c_int32), ("reserved", C.c_int32)]
+                ("tls_recovery", C.c_int32), ("static_check", C.c_int32)]
+
+
+class jp_static(C.Structure):
+    _fields_ = [("affine", C.c_int32), ("independent", C.c_int32), ("in_range", C.c_int32), ("reserved", C.c_int32),
+                ("alpha", C.c_int64 * 4), ("beta", C.c_int64 * 4)]
 
 
 class jp_sched_result(C.Structure):
@@ -83,6 +88,8 @@ SIGNATURES = [
     ("jp_profile_classify", _I32, [_P(jp_loop), _V, _SZ, _V, _I64, _V, _P(jp_profile), _V]),
     ("jp_profile_density", _I32, [_P(jp_loop), _V, _SZ, _V, _I64, _V, _P(jp_profile), _V]),
     ("jp_select_mode", _I32, [_P(jp_loop), _P(jp_profile), _D]),
+    ("jp_static_check", _I32, [_P(jp_loop), _V, _SZ, _P(jp_static), _V]),
+    ("jp_affine_dependence", _I32, [_I64, _I64, _I64, _I64, _I64]),
     ("jp_run_doall", _I32, [_P(jp_loop), _P(jp_profile), _V, _SZ, _V]),
     ("jp_run_privatized", _I32, [_P(jp_loop), _P(jp_profile), _V, _SZ, _V]),
     ("jp_priv_stream", _I32, [_P(jp_loop), _P(jp_profile), _V, _SZ, _I32, _V]),

@@ -350,6 +350,77 @@ int32_t jp_select_mode(const jp_loop *L, const jp_profile *p, double tau_high) {
   return select_mode_counts(p->n, p->raw_iters, p->war_iters, p->waw_iters, tau_high);
 }
 
+// ---------------------------------------------------------------------------
+// static analysis lite (jp_static.cu)
+// ---------------------------------------------------------------------------
+static jp_status static_check(const jp_loop *L, const Job &j, void *ws, const Layout &lo, jp_static *out,
+                              cudaStream_t st) {
+  memset(out, 0, sizeof *out);
+  int64_t *hdr = at<int64_t>(ws, lo, R_HEADER);
+  int *flags = reinterpret_cast<int *>(&hdr[H_AFFINE]);
+  JP_CUDA(launch_affine(j, flags, st), "affine");
+  const int32_t *ps[4] = {j.d.r, j.d.r2, j.d.w, j.d.s};
+  int32_t first[4][2] = {{0, 0}, {0, 0}, {0, 0}, {0, 0}};
+  for (int q = 0; q < 4; q++)
+    if (ps[q] && L->n > 0)
+      JP_CUDA(cudaMemcpyAsync(first[q], ps[q], L->n > 1 ? 8 : 4, cudaMemcpyDeviceToHost, st), "affine D2H");
+  int fl[4];
+  JP_CUDA(d2h_small_sync(fl, flags, sizeof fl, st), "affine D2H");
+  out->affine = 1;
+  for (int q = 0; q < 4; q++) {
+    if (ps[q]) {
+      out->affine &= fl[q] ? 1 : 0;
+      out->beta[q] = first[q][0];
+      out->alpha[q] = L->n > 1 ? (int64_t)first[q][1] - first[q][0] : 0;
+    } else {
+      out->alpha[q] = 1;
+      out->beta[q] = L->ident_off;
+    }
+  }
+  if (!out->affine) return JP_OK;
+  // accesses per array (SURVEY Sec.8 opcode table): 0 r, 1 r2, 2 w, 3 s
+  struct Acc { int q; bool write; int arr; };   // arr 0 A, 1 X, 2 T
+  Acc acc[4];
+  int na = 0;
+  switch (L->op) {
+    case JP_OP_ADD_C: acc[na++] = {2, true, 0}; acc[na++] = {0, false, 0}; break;
+    case JP_OP_SAXPY: acc[na++] = {2, true, 0}; acc[na++] = {0, false, 1}; break;     // Y[w] read == its write
+    case JP_OP_PRIV_TMP: acc[na++] = {3, true, 2}; acc[na++] = {2, true, 0}; acc[na++] = {0, false, 1}; break;
+    default: acc[na++] = {2, true, 0}; acc[na++] = {0, false, 0}; acc[na++] = {1, false, 0}; break;
+  }
+  const int64_t len[3] = {L->len_A, L->len_X, L->len_T};
+  out->in_range = 1;
+  for (int k = 0; k < na; k++) {
+    const Acc &a = acc[k];
+    if (L->n == 0) break;
+    const int64_t v0 = out->beta[a.q], v1 = out->beta[a.q] + out->alpha[a.q] * (L->n - 1);
+    if (std::min(v0, v1) < 0 || std::max(v0, v1) >= len[a.arr]) out->in_range = 0;
+  }
+  out->independent = 1;
+  for (int f = 0; f < na; f++) {
+    if (!acc[f].write) continue;
+    for (int g = 0; g < na; g++) {
+      if (acc[g].arr != acc[f].arr) continue;
+      if (affine_conflict(out->alpha[acc[f].q], out->beta[acc[f].q], out->alpha[acc[g].q], out->beta[acc[g].q], L->n))
+        out->independent = 0;
+    }
+  }
+  return JP_OK;
+}
+
+int32_t jp_affine_dependence(int64_t af, int64_t bf, int64_t ag, int64_t bg, int64_t n) {
+  return affine_conflict(af, bf, ag, bg, n) ? 1 : 0;
+}
+
+jp_status jp_static_check(const jp_loop *L, void *ws, size_t ws_bytes, jp_static *out, jp_stream_t st) {
+  JP_TRY(check_loop(L));
+  if (!out) return fail(JP_ERR_ARG, "result is NULL");
+  JP_TRY(need_device());
+  Layout lo;
+  JP_TRY(check_ws(L, ws, ws_bytes, 0, lo));
+  return static_check(L, make_job(L), ws, lo, out, (cudaStream_t)st);
+}
+
 jp_status jp_run_doall(const jp_loop *L, const jp_profile *p, void *ws, size_t ws_bytes, jp_stream_t stp) {
   JP_TRY(check_loop(L));
   if (p && (p->raw_iters || p->war_iters || p->waw_iters))
@@ -983,6 +1054,22 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
       res->tls_cluster = 1;
     }
     return JP_OK;
+  }
+  if (c.static_check == 0 && ws) {
+    // static analysis lite: affine, in-range, conflict-free -> DOALL without a profile
+    Layout ls;
+    JP_TRY(check_ws(L, ws, ws_bytes, 0, ls));
+    jp_static sa;
+    JP_TRY(static_check(L, j, ws, ls, &sa, st));
+    if (sa.independent && sa.in_range) {
+      res->mode = JP_MODE_DOALL;
+      res->profiled = 0;
+      res->n_tasks = 1;
+      res->n_batches = 1;
+      JP_CUDA(launch_doall(j, st), "doall");
+      res->task_mode_iters[JP_MODE_DOALL] = L->n;
+      return JP_OK;
+    }
   }
   jp_profile p;
   // the classify pass also writes the TLS guide bitmaps when the loop can be guided

@@ -70,6 +70,10 @@ cudaError_t launch_task_conflicts(const Job &j, const int32_t *chunk_task, int64
                                   unsigned long long *wmT, unsigned long long *rmT,
                                   unsigned long long *conf, cudaStream_t st);
 
+// static analysis lite (jp_static.cu): flags[q] = index array q (r, r2, w, s) is affine
+cudaError_t launch_affine(const Job &j, int *flags, cudaStream_t st);
+bool affine_conflict(int64_t af, int64_t bf, int64_t ag, int64_t bg, int64_t n);
+
 // tiny loops (jp_tiny.cu): the whole schedule in one CTA's shared memory
 bool tiny_eligible(const jp_loop *L);
 cudaError_t launch_tiny(const Job &j, const jp_loop *L, double tau, int64_t window, int64_t w_max, int recovery,
