@@ -52,7 +52,8 @@ typedef enum { JP_OP_ADD_C = 0, JP_OP_SAXPY = 1, JP_OP_PRIV_TMP = 2, JP_OP_STENC
 typedef enum { JP_MODE_DOALL = 0, JP_MODE_PRIVATIZED = 1, JP_MODE_TLS = 2,
                JP_MODE_SEQ_RECOMMENDED = 3 } jp_mode;
 /* scheme(s) clause, Table I: sharing (default) or stealing (Sec. V). */
-typedef enum { JP_SCHED_SHARING = 0, JP_SCHED_STEALING = 1 } jp_scheme;
+/* JP_SCHED_AUTO: for workflows (jp_schedule_workflow) only -- Sec. V.C. */
+typedef enum { JP_SCHED_SHARING = 0, JP_SCHED_STEALING = 1, JP_SCHED_AUTO = 2 } jp_scheme;
 
 typedef union { int32_t i; float f; } jp_scalar;
 
@@ -327,6 +328,41 @@ jp_status jp_plan_stealing(const int64_t *tasks, int64_t n_tasks, int32_t world,
                            int64_t chunk_iters, const double *speed, double speed_tls,
                            int64_t *chunks /* host [cap][4]: start,end,mode,owner */,
                            int64_t cap, int64_t *n_out, int64_t *stolen_out);
+
+/* ---- workflows: several loops and their PDG (P:L197-200
+ * "dependencies between loops are also represented by the program dependency
+ * graph", Alg. 1 and P:L438-460 "a task or job refers to a loop and the PDG
+ * gives us a workflow", P:L461-469 scheme selection; readings B9, B10) ------
+ * Loop u depends on an earlier loop t iff a byte of device memory is written by
+ * one of them and read or written by the other (arrays are the ranges
+ * [ptr, ptr + 4*len) of A, X, T and the index arrays; A is read by ADD_C,
+ * SAXPY and STENCIL2, T and A are written).  batch[u] = 1 + max batch of its
+ * dependencies (0 if none): each batch is a set of data-independent loops.
+ * scheme AUTO resolves to STEALING when some batch holds >= 2 loops and no
+ * loop carries more than half of all iterations ("computations evenly
+ * distributed across several data-independent loops"), else SHARING
+ * ("heavy computations centralized in only one or few loops").  host only.   */
+#define JP_MAX_LOOPS 64
+typedef struct {
+  int32_t scheme;               /* the scheme the workflow runs with (AUTO resolved) */
+  int32_t n_batches;
+  int32_t batch[JP_MAX_LOOPS];  /* topological level of each loop                    */
+  uint64_t deps[JP_MAX_LOOPS];  /* bit t of deps[u]: loop u depends on loop t < u     */
+} jp_workflow_plan;
+jp_status jp_plan_workflow(const jp_loop *loops /* host [n] */, int32_t n, int32_t scheme,
+                           jp_workflow_plan *out /* host */);
+/* Runs a workflow on the current device: SHARING executes the loops in
+ * program order, each through jp_schedule with the whole device; STEALING
+ * executes batch after batch, the loops of a batch concurrently on separate
+ * streams (each through jp_schedule on its own workspace).  cfg->scheme picks
+ * the workflow scheme (AUTO allowed); every other cfg field applies to each
+ * loop, which runs with the single-loop scheme SHARING.  ws / ws_bytes (host
+ * arrays [n]): one workspace per loop (NULL entries: loops that need none).
+ * res (host [n]): each loop's jp_sched_result.  syncs.                       */
+jp_status jp_schedule_workflow(const jp_loop *loops /* host [n] */, int32_t n, const jp_sched_cfg *cfg,
+                               void *const *ws /* host [n] */, const size_t *ws_bytes /* host [n] */,
+                               jp_sched_result *res /* host [n] */, jp_workflow_plan *plan /* host */,
+                               jp_stream_t st);
 
 /* Apply packed last-writer keys: arr[a] = keys[a] ? lo32(keys[a]) : arr[a]. */
 jp_status jp_merge_apply(void *arr, int64_t len, const int64_t *keys, jp_stream_t st);

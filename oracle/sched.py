@@ -99,3 +99,33 @@ def stealing_plan(tasks, world, chunk, speed=None, speed_tls=1.0):
         chunks[c][4] = k
         clock[k] += (chunks[c][1] - chunks[c][0]) / rate
     return [(c[0], c[1], c[2], c[4]) for c in chunks], stolen
+
+
+# ---------------------------------------------------------------------------
+# workflows (P:L197-200 PDG, Alg. 1 over loops, P:L461-469 scheme
+# selection; readings B9, B10)
+# ---------------------------------------------------------------------------
+SHARING, STEALING, AUTO = 0, 1, 2
+
+
+def workflow_plan(footprints, iters, scheme=AUTO):
+    """footprints[u]: list of (lo, hi, writes) byte ranges loop u touches; iters[u]
+    its trip count.  Loop u depends on t < u iff a range of one that writes
+    overlaps a range of the other; batch[u] = 1 + max batch of its dependencies.
+    AUTO -> STEALING iff some batch holds >= 2 loops and no loop has more than
+    half of all iterations, else SHARING."""
+    n = len(footprints)
+    batch = [0] * n
+    deps = [0] * n
+    for u in range(n):
+        for t in range(u):
+            hit = any((wa or wb) and la < hb and lb < ha
+                      for (la, ha, wa) in footprints[t] for (lb, hb, wb) in footprints[u])
+            if hit:
+                deps[u] |= 1 << t
+                batch[u] = max(batch[u], batch[t] + 1)
+    n_batches = max(batch) + 1 if n else 0
+    if scheme == AUTO:
+        wide = any(batch.count(b) >= 2 for b in range(n_batches))
+        scheme = STEALING if wide and 2 * max(iters, default=0) <= sum(iters) else SHARING
+    return {"scheme": scheme, "n_batches": n_batches, "batch": batch, "deps": deps}

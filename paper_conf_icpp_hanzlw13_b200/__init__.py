@@ -16,7 +16,7 @@ from . import _abi
 from ._abi import (  # noqa: F401
     JP_I32, JP_F32, JP_OP_ADD_C, JP_OP_SAXPY, JP_OP_PRIV_TMP, JP_OP_STENCIL2,
     JP_MODE_DOALL, JP_MODE_PRIVATIZED, JP_MODE_TLS, JP_MODE_SEQ_RECOMMENDED, MODE_NAMES,
-    JP_SCHED_SHARING, JP_SCHED_STEALING, JP_TLS_RESTART, JP_TLS_ONCHIP, JP_WS_PROFILE, JP_WS_PRIV, JP_WS_TLS, JP_WS_SCHED, JP_WS_GUIDE, JP_WS_ALL,
+    JP_SCHED_SHARING, JP_SCHED_STEALING, JP_SCHED_AUTO, JP_TLS_RESTART, JP_TLS_ONCHIP, JP_WS_PROFILE, JP_WS_PRIV, JP_WS_TLS, JP_WS_SCHED, JP_WS_GUIDE, JP_WS_ALL,
     REGIONS, JPError, check, lib,
 )
 
@@ -264,6 +264,32 @@ def jp_schedule(loop: Loop, ws=None, cfg=None, stream=None, **kw) -> dict:
     p, nb = _ws(ws)
     check(lib().jp_schedule(loop.ref, C.byref(cfg), p, nb, C.byref(res), _stream(stream)))
     return _res_dict(res)
+
+
+def _plan_dict(p: _abi.jp_workflow_plan, n: int) -> dict:
+    return {"scheme": p.scheme, "n_batches": p.n_batches, "batch": list(p.batch[:n]), "deps": list(p.deps[:n])}
+
+
+def jp_plan_workflow(loops, scheme=JP_SCHED_AUTO) -> dict:
+    """PDG batches of a workflow of loops (host only; readings B9, B10)."""
+    arr = (_abi.jp_loop * max(len(loops), 1))(*[lp.c for lp in loops])
+    out = _abi.jp_workflow_plan()
+    check(lib().jp_plan_workflow(arr, len(loops), int(scheme), C.byref(out)))
+    return _plan_dict(out, len(loops))
+
+
+def jp_schedule_workflow(loops, wss=None, cfg=None, stream=None, **kw):
+    """Run a workflow (list of Loop) with one workspace per loop; returns (results, plan)."""
+    cfg = cfg if cfg is not None else sched_cfg(**kw)
+    n = len(loops)
+    arr = (_abi.jp_loop * max(n, 1))(*[lp.c for lp in loops])
+    wss = wss if wss is not None else [None] * n
+    wp = (C.c_void_p * max(n, 1))(*[None if w is None else w.data_ptr() for w in wss])
+    wb = (C.c_size_t * max(n, 1))(*[0 if w is None else w.numel() for w in wss])
+    res = (_abi.jp_sched_result * max(n, 1))()
+    plan = _abi.jp_workflow_plan()
+    check(lib().jp_schedule_workflow(arr, n, C.byref(cfg), wp, wb, res, C.byref(plan), _stream(stream)))
+    return [_res_dict(res[u]) for u in range(n)], _plan_dict(plan, n)
 
 
 def jp_stage_bytes(loop: Loop) -> int:

@@ -22,7 +22,8 @@ JP_I32, JP_F32 = 0, 1
 JP_OP_ADD_C, JP_OP_SAXPY, JP_OP_PRIV_TMP, JP_OP_STENCIL2 = 0, 1, 2, 3
 JP_MODE_DOALL, JP_MODE_PRIVATIZED, JP_MODE_TLS, JP_MODE_SEQ_RECOMMENDED = 0, 1, 2, 3
 MODE_NAMES = {0: "DOALL", 1: "PRIVATIZED", 2: "TLS", 3: "SEQ_RECOMMENDED"}
-JP_SCHED_SHARING, JP_SCHED_STEALING = 0, 1
+JP_SCHED_SHARING, JP_SCHED_STEALING, JP_SCHED_AUTO = 0, 1, 2
+JP_MAX_LOOPS = 64
 JP_TLS_RESTART, JP_TLS_ONCHIP = 0, 1
 JP_WS_PROFILE, JP_WS_PRIV, JP_WS_TLS, JP_WS_SCHED, JP_WS_GUIDE, JP_WS_ALL = 1, 2, 4, 8, 16, 31
 REGIONS = {"header": 0, "minW_A": 1, "minR_A": 2, "minW_T": 3, "minR_T": 4, "keys_A": 5, "keys_T": 6,
@@ -71,6 +72,10 @@ class jp_static(C.Structure):
                 ("alpha", C.c_int64 * 4), ("beta", C.c_int64 * 4)]
 
 
+class jp_workflow_plan(C.Structure):
+    _fields_ = [("scheme", C.c_int32), ("n_batches", C.c_int32), ("batch", C.c_int32 * 64), ("deps", C.c_uint64 * 64)]
+
+
 class jp_sched_result(C.Structure):
     _fields_ = [("mode", C.c_int32), ("profiled", C.c_int32), ("prof", jp_profile), ("tls", jp_tls_stats),
                 ("n_tasks", C.c_int64), ("n_batches", C.c_int64), ("task_mode_iters", C.c_int64 * 4),
@@ -102,6 +107,9 @@ SIGNATURES = [
     ("jp_schedule_host", _I32, [_P(jp_loop), _P(jp_sched_cfg), _V, _SZ, _V, _SZ, _P(jp_sched_result), _V]),
     ("jp_plan_sharing", _I32, [_I64, _I32, _P(_D), _P(_I64)]),
     ("jp_plan_stealing", _I32, [_P(_I64), _I64, _I32, _I64, _P(_D), _D, _P(_I64), _I64, _P(_I64), _P(_I64)]),
+    ("jp_plan_workflow", _I32, [_P(jp_loop), _I32, _I32, _P(jp_workflow_plan)]),
+    ("jp_schedule_workflow", _I32, [_P(jp_loop), _I32, _P(jp_sched_cfg), _P(_V), _P(_SZ), _P(jp_sched_result),
+                                    _P(jp_workflow_plan), _V]),
     ("jp_merge_apply", _I32, [_V, _I64, _V, _V]),
     ("jp_last_error", C.c_char_p, []),
     ("jp_version", C.c_char_p, []),

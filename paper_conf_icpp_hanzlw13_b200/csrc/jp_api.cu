@@ -1095,6 +1095,121 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
   return run_mode(L, j, run, &p, c, ws, ws_bytes, res, st, gfuse && p.waw_iters == 0);
 }
 
+
+// ---------------------------------------------------------------------------
+// workflows: PDG of loops (readings B9, B10)
+// ---------------------------------------------------------------------------
+namespace {
+struct Span { uintptr_t lo, hi; bool write; };
+// the device memory a loop touches: index arrays and X read; A read (ADD_C,
+// SAXPY, STENCIL2) and written; T written (its covered reads are its own writes)
+static int footprint(const jp_loop *L, Span *out) {
+  int k = 0;
+  auto add = [&](const void *p, int64_t len, bool w) {
+    if (p && len > 0 && L->n > 0) out[k++] = {(uintptr_t)p, (uintptr_t)p + 4 * (uintptr_t)len, w};
+  };
+  add(L->r, L->n, false);
+  add(L->r2, L->n, false);
+  add(L->w, L->n, false);
+  add(L->s, L->n, false);
+  add(L->X, L->len_X, false);
+  if (L->op != JP_OP_PRIV_TMP) add(L->A, L->len_A, false);
+  add(L->A, L->len_A, true);
+  if (L->op == JP_OP_PRIV_TMP) add(L->T, L->len_T, true);
+  return k;
+}
+}  // namespace
+
+static jp_status plan_workflow(const jp_loop *loops, int32_t n, int32_t scheme, jp_workflow_plan *out) {
+  if (!loops || !out || n < 0 || n > JP_MAX_LOOPS) return fail(JP_ERR_ARG, "need 0 <= n <= %d loops", JP_MAX_LOOPS);
+  if (scheme < JP_SCHED_SHARING || scheme > JP_SCHED_AUTO) return fail(JP_ERR_ARG, "bad scheme %d", scheme);
+  memset(out, 0, sizeof *out);
+  std::vector<std::vector<Span>> fp(n);
+  for (int u = 0; u < n; u++) {
+    JP_TRY(check_loop(&loops[u]));
+    Span s[8];
+    fp[u].assign(s, s + footprint(&loops[u], s));
+  }
+  int64_t total = 0, biggest = 0;
+  for (int u = 0; u < n; u++) {
+    for (int t = 0; t < u; t++) {
+      bool dep = false;
+      for (const Span &a : fp[t])
+        for (const Span &b : fp[u])
+          dep = dep || ((a.write || b.write) && a.lo < b.hi && b.lo < a.hi);
+      if (dep) {
+        out->deps[u] |= 1ull << t;
+        out->batch[u] = std::max(out->batch[u], out->batch[t] + 1);
+      }
+    }
+    out->n_batches = std::max(out->n_batches, out->batch[u] + 1);
+    total += loops[u].n;
+    biggest = std::max(biggest, loops[u].n);
+  }
+  if (scheme == JP_SCHED_AUTO) {
+    bool wide = false;
+    for (int b = 0; b < out->n_batches && !wide; b++) {
+      int cnt = 0;
+      for (int u = 0; u < n; u++) cnt += out->batch[u] == b;
+      wide = cnt >= 2;
+    }
+    scheme = wide && 2 * biggest <= total ? JP_SCHED_STEALING : JP_SCHED_SHARING;
+  }
+  out->scheme = scheme;
+  return JP_OK;
+}
+
+jp_status jp_plan_workflow(const jp_loop *loops, int32_t n, int32_t scheme, jp_workflow_plan *out) {
+  return plan_workflow(loops, n, scheme, out);
+}
+
+jp_status jp_schedule_workflow(const jp_loop *loops, int32_t n, const jp_sched_cfg *cfgp, void *const *ws,
+                               const size_t *ws_bytes, jp_sched_result *res, jp_workflow_plan *plan,
+                               jp_stream_t stp) {
+  if (!res || !plan) return fail(JP_ERR_ARG, "result / plan is NULL");
+  JP_TRY(need_device());
+  jp_sched_cfg c = cfgp ? *cfgp : default_cfg();
+  JP_TRY(plan_workflow(loops, n, c.scheme, plan));
+  jp_sched_cfg lc = c;
+  lc.scheme = JP_SCHED_SHARING;   // each loop: the single-loop scheme
+  cudaStream_t st = (cudaStream_t)stp;
+  auto wsp = [&](int u) { return ws ? ws[u] : nullptr; };
+  auto wsb = [&](int u) { return ws_bytes ? ws_bytes[u] : (size_t)0; };
+  if (plan->scheme == JP_SCHED_SHARING) {
+    for (int u = 0; u < n; u++) JP_TRY(jp_schedule(&loops[u], &lc, wsp(u), wsb(u), &res[u], stp));
+    return JP_OK;
+  }
+  // STEALING on one device: batch after batch; the loops of a batch run
+  // concurrently, each on its own stream, joined before the next batch
+  cudaEvent_t ev0;
+  JP_CUDA(cudaEventCreateWithFlags(&ev0, cudaEventDisableTiming), "event");
+  std::vector<cudaEvent_t> evs;
+  jp_status status = JP_OK;
+  for (int b = 0; b < plan->n_batches && status == JP_OK; b++) {
+    cudaEventRecord(ev0, st);
+    std::vector<cudaEvent_t> joins;
+    int k = 0;
+    for (int u = 0; u < n && status == JP_OK; u++) {
+      if (plan->batch[u] != b) continue;
+      cudaStream_t s2 = g_pool.get(k++);
+      cudaStreamWaitEvent(s2, ev0, 0);
+      status = jp_schedule(&loops[u], &lc, wsp(u), wsb(u), &res[u], (jp_stream_t)s2);
+      cudaEvent_t e;
+      cudaEventCreateWithFlags(&e, cudaEventDisableTiming);
+      cudaEventRecord(e, s2);
+      joins.push_back(e);
+      evs.push_back(e);
+    }
+    for (auto e : joins) cudaStreamWaitEvent(st, e, 0);
+  }
+  cudaError_t ce = cudaStreamSynchronize(st);
+  for (auto e : evs) cudaEventDestroy(e);
+  cudaEventDestroy(ev0);
+  if (status != JP_OK) return status;
+  if (ce != cudaSuccess) return fail(JP_ERR_CUDA, "workflow: %s", cudaGetErrorString(ce));
+  return JP_OK;
+}
+
 // ---------------------------------------------------------------------------
 // host-buffer entry point (end-to-end: H2D, schedule, D2H)
 // ---------------------------------------------------------------------------

@@ -200,3 +200,49 @@ def config5(n: int = 1 << 24, density: float = 0.05, delta: int = 1024, device="
     return Workload("config5", 0, 0, n, i32_data(seed, 1, n, device), r=r.to(torch.int32), w=w.to(torch.int32),
                     c0=C0_I32, meta={"regions": [(0, h), (h, h + q), (h + q, n)], "raw": k,
                                      "war": q - 2, "waw": m, "delta": delta, "density": density})
+
+
+# ---------------------------------------------------------------------------
+# workflows of several loops: the shapes of the
+# paper's task-stealing applications.  Loops share storage through
+# tensor views, so the device ranges they read and write are those of the
+# original program.  Each function returns (loops, arrays): a list of
+# Workloads in program order and the distinct base tensors they view.
+# ---------------------------------------------------------------------------
+def workflow_bicg(n: int = 1 << 24, parts: int = 4, device="cpu"):
+    """BICG: two independent DOALL loops of similar work (s = c0*p + s and
+    t = c0*q + t, fp32), each divided evenly into `parts` subloops."""
+    seed = 1006
+    p, q = f32_data(seed, 1, n, device), f32_data(seed, 2, n, device)
+    s, t = f32_data(seed, 3, n, device), f32_data(seed, 4, n, device)
+    m = n // parts
+    loops = []
+    for X, Y in ((p, s), (q, t)):
+        for k in range(parts):
+            b, e = k * m, (n if k == parts - 1 else (k + 1) * m)
+            loops.append(Workload("bicg", 1, 1, e - b, Y[b:e], X=X[b:e], c0=C0_F32))
+    return loops, [p, q, s, t]
+
+
+def workflow_2mm(n: int = 1 << 24, device="cpu"):
+    """2MM: two DOALL loops, the second consuming the first's output
+    (y = c0*x + y, then z = c0*y + z, fp32)."""
+    seed = 1007
+    x, y, z = f32_data(seed, 1, n, device), f32_data(seed, 2, n, device), f32_data(seed, 3, n, device)
+    return [Workload("2mm-1", 1, 1, n, y, X=x, c0=C0_F32), Workload("2mm-2", 1, 1, n, z, X=y, c0=C0_F32)], [x, y, z]
+
+
+def workflow_crypt(n: int = 1 << 24, parts: int = 8, device="cpu"):
+    """Crypt: an encryption loop (c[i] = c0*p[pi(i)] + c[i], int32) and a
+    decryption loop reading the whole cipher (d[i] = c0*c[pi2(i)] + d[i]),
+    each divided evenly into `parts` subloops: 2*parts loops in two batches."""
+    seed = 1008
+    p, c, d = i32_data(seed, 1, n, device), i32_data(seed, 2, n, device), i32_data(seed, 3, n, device)
+    pi, pi2 = permutation(seed, n, device).to(torch.int32), permutation(seed + 1, n, device).to(torch.int32)
+    m = n // parts
+    loops = []
+    for X, Y, perm in ((p, c, pi), (c, d, pi2)):
+        for k in range(parts):
+            b, e = k * m, (n if k == parts - 1 else (k + 1) * m)
+            loops.append(Workload("crypt", 1, 0, e - b, Y[b:e], r=perm[b:e], X=X, c0=C0_I32))
+    return loops, [p, c, d, pi, pi2]
