@@ -323,6 +323,33 @@ def modes_sweep(jp, dev, st):
     out["config5_mixed"] = {"n": wl.n, "iters_per_s": wl.n / t, "ms": t * 1e3, "n_tasks": res["n_tasks"],
                             "n_batches": res["n_batches"], "task_mode_iters": res["task_mode_iters"],
                             "tls": res["tls"]}
+    del wl, ws, L, A0
+    # workflows: the paper's task-stealing shapes, N = 2^24
+    # iterations per original loop, every scheme; whole jp_schedule_workflow call
+    wf = {}
+    for name, fn in (("bicg", synth.workflow_bicg), ("2mm", synth.workflow_2mm), ("crypt", synth.workflow_crypt)):
+        loops, arrays = fn(device=dev)
+        init = [b.clone() for b in arrays]
+        Ls = [jp.Loop.from_workload(x) for x in loops]
+        wss = [jp.workspace(x) for x in Ls]
+        row = {"loops": len(loops), "iters": sum(x.n for x in loops)}
+        for sname, sch in (("sharing", jp.JP_SCHED_SHARING), ("stealing", jp.JP_SCHED_STEALING),
+                           ("auto", jp.JP_SCHED_AUTO)):
+            ts = []
+            for rep in range(3):
+                for b, b0 in zip(arrays, init):
+                    b.copy_(b0)
+                torch.cuda.synchronize()
+                t0 = time.perf_counter()
+                _, plan = jp.jp_schedule_workflow(Ls, wss, scheme=sch, stream=st)
+                torch.cuda.synchronize()
+                ts.append(time.perf_counter() - t0)
+            t = min(ts[1:])
+            row[sname] = {"ms": t * 1e3, "iters_per_s": row["iters"] / t, "n_batches": plan["n_batches"],
+                          "scheme": ["sharing", "stealing"][plan["scheme"]]}
+        wf[name] = row
+        del loops, arrays, init, Ls, wss
+    out["workflows"] = wf
     return out
 
 
