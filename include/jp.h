@@ -367,6 +367,47 @@ jp_status jp_schedule_workflow(const jp_loop *loops /* host [n] */, int32_t n, c
 /* Apply packed last-writer keys: arr[a] = keys[a] ? lo32(keys[a]) : arr[a]. */
 jp_status jp_merge_apply(void *arr, int64_t len, const int64_t *keys, jp_stream_t st);
 
+/* ---- owner-partitioned sparse exchange --------
+ * Building blocks for the "one exchange step" of partitioned loops with
+ * indirect writes: the whole-loop first-writer / first-reader tables of the
+ * profile (reading A1; C1) and the last-writer keys of the privatized write-
+ * back (reading A9; C4) are per-address MAX reductions over the
+ * ranks.  Instead of all-reducing the dense tables, a rank packs the entries
+ * it touched into rows bucketed by the address's OWNER rank
+ * (owner(a) = a / ceil(len / world)), the caller all_to_alls them, and the
+ * owner folds them into its slice (the library never calls NCCL).
+ *
+ * A table is a dense device array of len elements of elem_bytes: 4 (int32,
+ * compared signed; len <= INT32_MAX) or 8 (uint64, compared unsigned).  One or
+ * two tables of the same length travel together (t1 NULL: one).  A row is
+ * 1 + ntab elements of elem_bytes, row-major: column 0 the address, then the
+ * value of each table at that address.                                       */
+
+/* Scratch (device, caller-owned, 8-byte aligned) jp_sparse_pack needs.       */
+size_t jp_sparse_scratch_bytes(int64_t len, int32_t world);
+/* Rows for every address a in [lo, hi) where t0[a] != empty or
+ * t1[a] != empty, in increasing address order -- hence grouped by owner --
+ * written to rows[0 .. m) (m = sum of counts).  counts (host [world]):
+ * number of rows of each owner (owners computed over the whole [0, len)).
+ * cap: capacity of rows in rows; when m > cap nothing beyond cap is written
+ * and JP_ERR_ARG is returned with counts filled.  syncs.                     */
+jp_status jp_sparse_pack(const void *t0, const void *t1 /* nullable */, int32_t elem_bytes, int64_t len,
+                         int64_t lo, int64_t hi, int64_t empty, int32_t world, void *rows, int64_t cap,
+                         int64_t *counts /* host [world] */, void *scratch, size_t scratch_bytes, jp_stream_t st);
+/* For each of the m rows: t_q[addr] = max(t_q[addr], row value q), atomic,
+ * in any order (MAX is order-free).  Rows with addr outside [0, len) are
+ * ignored (padding).                                                          */
+jp_status jp_sparse_reduce_max(void *t0, void *t1 /* nullable */, int32_t elem_bytes, int64_t len, const void *rows,
+                               int64_t m, jp_stream_t st);
+/* For each row (in place): row value q = t_q[addr]; out-of-range rows are left as they are. */
+jp_status jp_sparse_gather(const void *t0, const void *t1 /* nullable */, int32_t elem_bytes, int64_t len, void *rows,
+                           int64_t m, jp_stream_t st);
+/* For each row: t_q[addr] = row value q.  Rows must carry distinct addresses
+ * (as pack produces them; otherwise which row lands is unspecified);
+ * out-of-range rows are ignored.                                              */
+jp_status jp_sparse_scatter(void *t0, void *t1 /* nullable */, int32_t elem_bytes, int64_t len, const void *rows,
+                            int64_t m, jp_stream_t st);
+
 const char *jp_last_error(void);
 const char *jp_version(void);
 /* Number of kernels this library has launched in this process (for bench.py). */

@@ -24,7 +24,9 @@ __all__ = [
     "Loop", "workspace", "jp_workspace_bytes", "jp_ws_region", "jp_validate", "jp_profile_stamp",
     "jp_profile_classify", "jp_profile_density", "jp_select_mode", "jp_run_doall", "jp_run_privatized",
     "jp_priv_stream", "jp_priv_finalize", "jp_doall_kernel", "jp_tls_guide", "tls_first_window", "jp_run_tls", "jp_schedule", "jp_stage_bytes", "jp_schedule_host",
-    "jp_plan_sharing", "jp_plan_stealing", "jp_merge_apply", "jp_last_error", "jp_version", "jp_launch_count",
+    "jp_plan_sharing", "jp_plan_stealing", "jp_merge_apply",
+    "jp_sparse_scratch_bytes", "jp_sparse_pack", "jp_sparse_reduce_max", "jp_sparse_gather", "jp_sparse_scatter",
+    "jp_last_error", "jp_version", "jp_launch_count",
 ]
 
 _EL = {JP_I32: torch.int32, JP_F32: torch.float32}
@@ -328,6 +330,49 @@ def jp_plan_stealing(tasks, world: int, chunk_iters: int, speed=None, speed_tls:
 
 def jp_merge_apply(arr: torch.Tensor, keys: torch.Tensor, stream=None):
     check(lib().jp_merge_apply(arr.data_ptr(), arr.numel(), keys.data_ptr(), _stream(stream)))
+
+
+# ---- owner-partitioned sparse exchange (jp.h, NEXT-2) ----------------------
+def _tables(t0, t1):
+    if t0.dtype not in (torch.int32, torch.int64) or (t1 is not None and (t1.dtype != t0.dtype
+                                                                         or t1.numel() != t0.numel())):
+        raise ValueError("sparse tables: one or two int32 / int64 tensors of the same length")
+    return t0.element_size(), t0.numel(), 2 + (t1 is not None)   # row width: address + values
+
+
+def jp_sparse_scratch_bytes(length: int, world: int) -> int:
+    return int(lib().jp_sparse_scratch_bytes(int(length), int(world)))
+
+
+def jp_sparse_pack(t0: torch.Tensor, t1=None, empty: int = -1, world: int = 1, lo: int = 0, hi=None, stream=None):
+    """Rows [m, 1 + ntab] (t0's dtype; column 0 the address) of the entries of
+    [lo, hi) where a table is not ``empty``, sorted by address, and the per-owner
+    row counts (list of ``world`` ints)."""
+    eb, n, w = _tables(t0, t1)
+    hi = n if hi is None else int(hi)
+    cap = max(hi - int(lo), 0)
+    rows = torch.empty((max(cap, 1), w), dtype=t0.dtype, device=t0.device)
+    scratch = torch.empty(max(jp_sparse_scratch_bytes(n, world) // 8, 1), dtype=torch.int64, device=t0.device)
+    counts = (C.c_int64 * int(world))()
+    check(lib().jp_sparse_pack(t0.data_ptr(), _ptr(t1), eb, n, int(lo), hi, int(empty), int(world), rows.data_ptr(),
+                               cap, counts, scratch.data_ptr(), scratch.numel() * 8, _stream(stream)))
+    cl = list(counts)
+    return rows[:sum(cl)], cl
+
+
+def jp_sparse_reduce_max(t0: torch.Tensor, t1, rows: torch.Tensor, stream=None):
+    eb, n, _ = _tables(t0, t1)
+    check(lib().jp_sparse_reduce_max(t0.data_ptr(), _ptr(t1), eb, n, rows.data_ptr(), rows.shape[0], _stream(stream)))
+
+
+def jp_sparse_gather(t0: torch.Tensor, t1, rows: torch.Tensor, stream=None):
+    eb, n, _ = _tables(t0, t1)
+    check(lib().jp_sparse_gather(t0.data_ptr(), _ptr(t1), eb, n, rows.data_ptr(), rows.shape[0], _stream(stream)))
+
+
+def jp_sparse_scatter(t0: torch.Tensor, t1, rows: torch.Tensor, stream=None):
+    eb, n, _ = _tables(t0, t1)
+    check(lib().jp_sparse_scatter(t0.data_ptr(), _ptr(t1), eb, n, rows.data_ptr(), rows.shape[0], _stream(stream)))
 
 
 def jp_last_error() -> str:

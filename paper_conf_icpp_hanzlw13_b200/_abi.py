@@ -111,6 +111,11 @@ SIGNATURES = [
     ("jp_schedule_workflow", _I32, [_P(jp_loop), _I32, _P(jp_sched_cfg), _P(_V), _P(_SZ), _P(jp_sched_result),
                                     _P(jp_workflow_plan), _V]),
     ("jp_merge_apply", _I32, [_V, _I64, _V, _V]),
+    ("jp_sparse_scratch_bytes", _SZ, [_I64, _I32]),
+    ("jp_sparse_pack", _I32, [_V, _V, _I32, _I64, _I64, _I64, _I64, _I32, _V, _I64, _P(_I64), _V, _SZ, _V]),
+    ("jp_sparse_reduce_max", _I32, [_V, _V, _I32, _I64, _V, _I64, _V]),
+    ("jp_sparse_gather", _I32, [_V, _V, _I32, _I64, _V, _I64, _V]),
+    ("jp_sparse_scatter", _I32, [_V, _V, _I32, _I64, _V, _I64, _V]),
     ("jp_last_error", C.c_char_p, []),
     ("jp_version", C.c_char_p, []),
     ("jp_launch_count", _I64, []),

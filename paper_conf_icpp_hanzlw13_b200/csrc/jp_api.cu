@@ -655,6 +655,73 @@ jp_status jp_merge_apply(void *arr, int64_t len, const int64_t *keys, jp_stream_
 }
 
 // ---------------------------------------------------------------------------
+// owner-partitioned sparse exchange (NEXT-2)
+// ---------------------------------------------------------------------------
+static jp_status check_sparse(const void *t0, int32_t elem, int64_t len, const void *rows, int64_t m) {
+  if (elem != 4 && elem != 8) return fail(JP_ERR_ARG, "elem_bytes must be 4 or 8 (got %d)", elem);
+  if (len < 0 || (elem == 4 && len > INT32_MAX)) return fail(JP_ERR_ARG, "bad table length %lld", (long long)len);
+  if (m < 0) return fail(JP_ERR_ARG, "negative row count");
+  if (m > 0 && (!t0 || !rows)) return fail(JP_ERR_ARG, "NULL table or rows");
+  return JP_OK;
+}
+
+size_t jp_sparse_scratch_bytes(int64_t len, int32_t world) {
+  if (len < 0 || world <= 0) return 0;
+  return sparse_scratch_bytes(len, world);
+}
+
+jp_status jp_sparse_pack(const void *t0, const void *t1, int32_t elem_bytes, int64_t len, int64_t lo, int64_t hi,
+                         int64_t empty, int32_t world, void *rows, int64_t cap, int64_t *counts, void *scratch,
+                         size_t scratch_bytes, jp_stream_t st) {
+  JP_TRY(check_sparse(t0, elem_bytes, len, rows, 0));
+  if (world <= 0 || !counts) return fail(JP_ERR_ARG, "world must be > 0 and counts non-NULL");
+  if (lo < 0 || hi < lo || hi > len) return fail(JP_ERR_ARG, "bad range [%lld, %lld) of a %lld-entry table",
+                                                 (long long)lo, (long long)hi, (long long)len);
+  if (cap < 0 || (cap > 0 && !rows)) return fail(JP_ERR_ARG, "bad rows / cap");
+  if (hi > lo && !t0) return fail(JP_ERR_ARG, "NULL table");
+  const size_t need = sparse_scratch_bytes(len, world);
+  if (!scratch || scratch_bytes < need || ((uintptr_t)scratch & 7))
+    return fail(JP_ERR_WORKSPACE, "sparse scratch of %zu bytes (8-byte aligned) needed", need);
+  JP_TRY(need_device());
+  for (int k = 0; k < world; k++) counts[k] = 0;
+  if (hi == lo) return JP_OK;
+  const cudaStream_t s = (cudaStream_t)st;
+  const int64_t tiles = sparse_pack_tiles(len, lo, hi, world);
+  int64_t *counts_dev = static_cast<int64_t *>(scratch) + 2 * tiles + 1;
+  JP_CUDA(launch_sparse_pack(t0, t1, elem_bytes, len, lo, hi, empty, world, rows, cap, counts_dev, scratch, s),
+          "sparse pack");
+  JP_CUDA(d2h_small_sync(counts, counts_dev, sizeof(int64_t) * world, s), "sparse pack D2H");
+  int64_t m = 0;
+  for (int k = 0; k < world; k++) m += counts[k];
+  if (m > cap) return fail(JP_ERR_ARG, "%lld rows do not fit the %lld-row buffer", (long long)m, (long long)cap);
+  return JP_OK;
+}
+
+static jp_status sparse_rows(void *t0, void *t1, int32_t elem, int64_t len, void *rows, int64_t m, int what,
+                             jp_stream_t st, const char *where) {
+  JP_TRY(check_sparse(t0, elem, len, rows, m));
+  JP_TRY(need_device());
+  JP_CUDA(launch_sparse_rows(t0, t1, elem, len, rows, m, what, (cudaStream_t)st), where);
+  return JP_OK;
+}
+
+jp_status jp_sparse_reduce_max(void *t0, void *t1, int32_t elem_bytes, int64_t len, const void *rows, int64_t m,
+                               jp_stream_t st) {
+  return sparse_rows(t0, t1, elem_bytes, len, const_cast<void *>(rows), m, 0, st, "sparse reduce");
+}
+
+jp_status jp_sparse_gather(const void *t0, const void *t1, int32_t elem_bytes, int64_t len, void *rows, int64_t m,
+                           jp_stream_t st) {
+  return sparse_rows(const_cast<void *>(t0), const_cast<void *>(t1), elem_bytes, len, rows, m, 1, st,
+                     "sparse gather");
+}
+
+jp_status jp_sparse_scatter(void *t0, void *t1, int32_t elem_bytes, int64_t len, const void *rows, int64_t m,
+                            jp_stream_t st) {
+  return sparse_rows(t0, t1, elem_bytes, len, const_cast<void *>(rows), m, 2, st, "sparse scatter");
+}
+
+// ---------------------------------------------------------------------------
 // plans (host only)
 // ---------------------------------------------------------------------------
 jp_status jp_plan_sharing(int64_t n, int32_t world, const double *weights, int64_t *ranges) {

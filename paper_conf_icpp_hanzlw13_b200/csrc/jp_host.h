@@ -62,6 +62,15 @@ cudaError_t launch_priv_stream(const Job &j, void *ws, const Layout &lo, bool cl
                                cudaStream_t st, int max_ctas = 0, bool fuse_apply = false, bool *applied = nullptr);
 cudaError_t launch_priv_finalize(const Job &j, void *ws, const Layout &lo, cudaStream_t st);
 cudaError_t launch_merge_apply(void *arr, int64_t len, const int64_t *keys, cudaStream_t st);
+// owner-partitioned sparse exchange (jp_exchange.cu)
+size_t sparse_scratch_bytes(int64_t len, int world);
+int64_t sparse_pack_tiles(int64_t len, int64_t lo, int64_t hi, int world);
+cudaError_t launch_sparse_pack(const void *t0, const void *t1, int elem, int64_t len, int64_t lo, int64_t hi,
+                               int64_t empty, int world, void *rows, int64_t cap, int64_t *counts_dev, void *scratch,
+                               cudaStream_t st);
+// what: 0 reduce max, 1 gather, 2 scatter
+cudaError_t launch_sparse_rows(void *t0, void *t1, int elem, int64_t len, void *rows, int64_t m, int what,
+                               cudaStream_t st);
 // STEALING scheduler helpers (jp_sched.cu): per-task write/read bitmasks of every
 // address, then the task x task conflict matrix conf[t] (bit u set: t and u
 // touch a common address and at least one of them writes it).

@@ -14,6 +14,23 @@ libjp.so and lets the kernels consume the results.  Collectives used
   bcast                      of the in/out array after a TLS run (TLS windows
       stay ordered on one GPU: "replicas only", north_star).
 
+``exchange="owner"`` replaces the dense C1 / C4
+all_reduces of len-sized tables by an owner-partitioned sparse exchange
+(jp_sparse_* in jp.h; owner(a) = a / ceil(len/world)):
+
+  C1o  pack the touched (addr, minW, minR) rows by owner -> all_to_all -> the
+       owner folds them (MAX) -> answers each row with the folded value ->
+       all_to_all back -> scatter.  Every address a rank's classify looks up is
+       one it touched, so it ends with exactly the dense all_reduce's values
+       there;
+  C4o  pack the nonzero (addr, key) rows by owner -> all_to_all -> the owner
+       folds them -> all_gather of each owner's final nonzero rows (padded
+       with address -1) -> scatter: every replica holds the merged keys.
+
+The bytes moved scale with the addresses the loop touches, not with len.
+Tables shorter than OWNER_MIN_LEN (e.g. the 1024-slot T of config 4) stay on
+the dense all_reduce.
+
 Iteration ranges come from ``jp_plan_sharing`` (boundary formula)
 and ``jp_plan_stealing`` (Alg. 1).  Every compute step is a
 libjp.so kernel; ``engine`` exists only so that the CPU tests can drive the
@@ -52,18 +69,85 @@ def _region(ws: torch.Tensor, loop, name: str, dtype, engine=None):
     return ws[off:off + nb].view(dtype)
 
 
-def profile_partitioned(loop, ws, group=None, engine=None) -> dict:
+OWNER_MIN_LEN = 1 << 16
+
+
+def _a2a_rows(rows, counts, group):
+    """all_to_all of owner-bucketed rows; returns (received rows, received counts)."""
+    sc = torch.tensor(counts, dtype=torch.int64, device=rows.device)
+    rc = torch.empty_like(sc)
+    dist.all_to_all_single(rc, sc, group=group)
+    rcl = [int(x) for x in rc.tolist()]
+    recv = rows.new_empty((sum(rcl), rows.shape[1]))
+    dist.all_to_all_single(recv, rows.contiguous(), output_split_sizes=rcl, input_split_sizes=list(counts),
+                           group=group)
+    return recv, rcl
+
+
+def owner_reduce_touched(t0, t1, empty, group=None, engine=None) -> dict:
+    """C1o: every entry this rank touched (t0 or t1 != empty) ends holding the MAX
+    over all ranks, as a dense all_reduce MAX would leave it there."""
+    jp = _engine(engine)
+    world, _ = world_rank(group)
+    rows, counts = jp.jp_sparse_pack(t0, t1, empty, world)
+    recv, rcl = _a2a_rows(rows, counts, group)
+    jp.jp_sparse_reduce_max(t0, t1, recv)
+    jp.jp_sparse_gather(t0, t1, recv)   # stream-ordered after every received row is folded
+    back = torch.empty_like(rows)
+    dist.all_to_all_single(back, recv, output_split_sizes=list(counts), input_split_sizes=rcl, group=group)
+    jp.jp_sparse_scatter(t0, t1, back)
+    return {"rows_sent": int(rows.shape[0]), "rows_recv": int(recv.shape[0]),
+            "bytes_sent": 2 * rows.numel() * rows.element_size()}
+
+
+def owner_reduce_replicate(t, empty, group=None, engine=None) -> dict:
+    """C4o: t ends, on every rank, equal to the all_reduce MAX of t over the ranks
+    at every address where some rank holds a non-empty entry."""
+    jp = _engine(engine)
+    world, rank = world_rank(group)
+    rows, counts = jp.jp_sparse_pack(t, None, empty, world)
+    recv, _ = _a2a_rows(rows, counts, group)
+    jp.jp_sparse_reduce_max(t, None, recv)
+    n = t.numel()
+    sl = -(-n // world)
+    fin, _ = jp.jp_sparse_pack(t, None, empty, 1, min(rank * sl, n), min((rank + 1) * sl, n))
+    m = torch.tensor([fin.shape[0]], dtype=torch.int64, device=t.device)
+    ms = [torch.empty_like(m) for _ in range(world)]
+    dist.all_gather(ms, m, group=group)
+    mx = max(int(x.item()) for x in ms)
+    pad = torch.full((max(mx, 1), 2), -1, dtype=t.dtype, device=t.device)
+    pad[:fin.shape[0]] = fin
+    got = [torch.empty_like(pad) for _ in range(world)]
+    dist.all_gather(got, pad, group=group)
+    jp.jp_sparse_scatter(t, None, torch.cat(got))
+    return {"rows_sent": int(rows.shape[0]) + world * pad.shape[0], "rows_recv": int(recv.shape[0]),
+            "bytes_sent": (rows.numel() + world * pad.numel()) * t.element_size()}
+
+
+def _reduce_tables(tabs, empty, group, exchange, jp):
+    """MAX of each table across the ranks: dense all_reduce, or the owner form."""
+    tabs = [t for t in tabs if t is not None]
+    if exchange == "owner" and tabs and tabs[0].numel() >= OWNER_MIN_LEN:
+        return tabs
+    for t in tabs:
+        dist.all_reduce(t, op=dist.ReduceOp.MAX, group=group)
+    return []
+
+
+def profile_partitioned(loop, ws, group=None, engine=None, exchange: str = "dense") -> dict:
     """Profile of the whole loop from rank-local ranges (iter_base = global id of
-    the rank's first iteration): stamp locally, C1, classify locally, C3.  The
-    result equals the single-GPU profile exactly (tested)."""
+    the rank's first iteration): stamp locally, C1 (dense or owner form),
+    classify locally, C3.  The result equals the single-GPU profile exactly
+    (tested)."""
     jp = _engine(engine)
     world, _ = world_rank(group)
     jp.jp_profile_stamp(loop, ws)
     if world > 1:
-        for name in ("minW_A", "minR_A", "minW_T", "minR_T"):
-            t = _region(ws, loop, name, torch.int32, jp)
-            if t is not None:
-                dist.all_reduce(t, op=dist.ReduceOp.MAX, group=group)
+        left = _reduce_tables([_region(ws, loop, n, torch.int32, jp) for n in ("minW_A", "minR_A")], -1, group,
+                              exchange, jp)
+        if left:
+            owner_reduce_touched(left[0], left[1] if len(left) > 1 else None, -1, group, jp)
+        _reduce_tables([_region(ws, loop, n, torch.int32, jp) for n in ("minW_T", "minR_T")], -1, group, "dense", jp)
     p = jp.jp_profile_classify(loop, ws)
     if world > 1:
         dev = ws.device
@@ -80,7 +164,7 @@ def profile_partitioned(loop, ws, group=None, engine=None) -> dict:
     return p
 
 
-def privatized_partitioned(loop, ws, prof, group=None, engine=None):
+def privatized_partitioned(loop, ws, prof, group=None, engine=None, exchange: str = "dense"):
     """PE(V) over rank-local ranges: keys locally, C4 (MAX over packed keys), then
     every rank applies the merged keys -- each rank ends with the sequential
     result in its replica of the keyed arrays; identity-indexed outputs stay
@@ -90,14 +174,13 @@ def privatized_partitioned(loop, ws, prof, group=None, engine=None):
     jp.jp_priv_stream(loop, prof, ws, clear_keys=True)
     if world > 1:
         for name in ("keys_A", "keys_T"):
-            t = _region(ws, loop, name, torch.int64, jp)
-            if t is not None:
-                dist.all_reduce(t, op=dist.ReduceOp.MAX, group=group)
+            for t in _reduce_tables([_region(ws, loop, name, torch.int64, jp)], 0, group, exchange, jp):
+                owner_reduce_replicate(t, 0, group, jp)
     jp.jp_priv_finalize(loop, ws)
 
 
 def schedule_partitioned(loop, ws, group=None, tau_high: float = 0.25, tls_window: int = 0, tls_w_max: int = 2048,
-                         full_loop=None, engine=None) -> dict:
+                         full_loop=None, engine=None, exchange: str = "dense") -> dict:
     """Task sharing of one loop across the ranks (P:L342-358 generalised to k
     devices).  ``loop`` is this rank's range (iter_base = its first global id,
     index arrays offset, element arrays shared-address replicas).
@@ -109,6 +192,7 @@ def schedule_partitioned(loop, ws, group=None, tau_high: float = 0.25, tls_windo
         dependence-free special case of PE(V));
         TLS / SEQ_RECOMMENDED: rank 0 runs the windows over ``full_loop`` and
         broadcasts the in/out arrays (replicas only).
+    ``exchange``: "dense" (all_reduce of the tables) or "owner" (NEXT-2).
     """
     jp = _engine(engine)
     world, rank = world_rank(group)
@@ -117,11 +201,13 @@ def schedule_partitioned(loop, ws, group=None, tau_high: float = 0.25, tls_windo
         res = jp.jp_schedule(loop, ws)
         res["scheme"] = "sharing"
         return res
-    prof = profile_partitioned(loop, ws, group, jp)
+    if exchange not in ("dense", "owner"):
+        raise ValueError(f"exchange must be 'dense' or 'owner', not {exchange!r}")
+    prof = profile_partitioned(loop, ws, group, jp, exchange)
     mode = jp.jp_select_mode(loop, prof, tau_high)
     res = {"mode": mode, "mode_name": _abi.MODE_NAMES[mode], "profiled": 1, "prof": prof, "scheme": "sharing"}
     if mode in (_abi.JP_MODE_DOALL, _abi.JP_MODE_PRIVATIZED):
-        privatized_partitioned(loop, ws, prof, group, jp)
+        privatized_partitioned(loop, ws, prof, group, jp, exchange)
     else:
         if full_loop is None:
             raise ValueError("TLS needs the whole loop on rank 0 (full_loop)")

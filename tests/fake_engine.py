@@ -181,3 +181,45 @@ def jp_run_tls(loop, window=0, w_max=65536, path=0, prof=None, ws=None, stats=Tr
     if loop.tensors["T"] is not None:
         _np(loop.tensors["T"])[:] = T
     return stats_
+
+
+# ---- owner-partitioned sparse exchange (jp.h jp_sparse_*), plain definitions ----
+def jp_sparse_pack(t0, t1=None, empty=-1, world=1, lo=0, hi=None):
+    n = t0.numel()
+    hi = n if hi is None else hi
+    a = np.arange(lo, hi, dtype=np.int64)
+    full = t0.numpy()[lo:hi] != empty
+    if t1 is not None:
+        full |= t1.numpy()[lo:hi] != empty
+    a = a[full]
+    cols = [a.astype(t0.numpy().dtype), t0.numpy()[a]] + ([t1.numpy()[a]] if t1 is not None else [])
+    rows = torch.from_numpy(np.stack(cols, axis=1).copy())
+    sl = max(-(-n // world), 1)
+    counts = [int(np.count_nonzero(a // sl == k)) for k in range(world)]
+    return rows, counts
+
+
+def _rows_ok(rows, n):
+    a = rows.numpy()[:, 0].astype(np.int64)
+    return a, (a >= 0) & (a < n)
+
+
+def jp_sparse_reduce_max(t0, t1, rows):
+    a, ok = _rows_ok(rows, t0.numel())
+    for q, t in enumerate([t0, t1]):
+        if t is not None:
+            np.maximum.at(t.numpy(), a[ok], rows.numpy()[ok, 1 + q])
+
+
+def jp_sparse_gather(t0, t1, rows):
+    a, ok = _rows_ok(rows, t0.numel())
+    for q, t in enumerate([t0, t1]):
+        if t is not None:
+            rows.numpy()[ok, 1 + q] = t.numpy()[a[ok]]
+
+
+def jp_sparse_scatter(t0, t1, rows):
+    a, ok = _rows_ok(rows, t0.numel())
+    for q, t in enumerate([t0, t1]):
+        if t is not None:
+            t.numpy()[a[ok]] = rows.numpy()[ok, 1 + q]

@@ -60,3 +60,15 @@ def bits_to_flags(raw_bits: torch.Tensor, n: int) -> np.ndarray:
     for k in range(n):
         out[k] = (b[k >> 5] >> (k & 31)) & 1
     return out
+
+
+def region_workload(wl, b: int, e: int, name: str = None):
+    """Iterations [b, e) of an indirect loop as a loop of its own (same arrays,
+    index arrays sliced), e.g. config 5's privatized tail or DOALL head."""
+    import synth
+    return synth.Workload(name or f"{wl.name}[{b}:{e}]", wl.op, wl.dtype, e - b, wl.A.clone(),
+                          r=None if wl.r is None else wl.r[b:e].clone(),
+                          r2=None if wl.r2 is None else wl.r2[b:e].clone(),
+                          w=None if wl.w is None else wl.w[b:e].clone(),
+                          s=None if wl.s is None else wl.s[b:e].clone(),
+                          X=wl.X, T=None if wl.T is None else wl.T.clone(), c0=wl.c0, c1=wl.c1)

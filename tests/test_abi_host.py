@@ -3,6 +3,7 @@ symbol include/jp.h declares, and its host-only logic (workspace layout, the
 Fig. 2(b) decision, the task-sharing / task-stealing plans) matches the plain
 restatements in oracle/sched.py.  No compute call is made without a GPU, except
 to check that one fails loudly with JP_ERR_CUDA (no CPU fallback)."""
+import ctypes as C
 import os
 import random
 import re
@@ -176,6 +177,31 @@ def test_compute_calls_fail_loudly_without_gpu():
     with pytest.raises(jp.JPError) as e:
         jp.jp_schedule(L, torch.zeros(1 << 20, dtype=torch.uint8))
     assert e.value.status == _abi.JP_ERR_CUDA
+    t = torch.zeros(100, dtype=torch.int32)
+    with pytest.raises(jp.JPError) as e:
+        jp.jp_sparse_pack(t, None, -1, 2)
+    assert e.value.status == _abi.JP_ERR_CUDA
+    with pytest.raises(jp.JPError) as e:
+        jp.jp_sparse_reduce_max(t, None, torch.zeros((3, 2), dtype=torch.int32))
+    assert e.value.status == _abi.JP_ERR_CUDA
+
+
+def test_sparse_exchange_bad_arguments():
+    """Argument errors of the NEXT-2 entry points are decided on the host."""
+    lib = _abi.lib()
+    cnt = (C.c_int64 * 2)()
+    buf = C.create_string_buffer(1 << 12)
+    p = C.addressof(buf)
+    assert lib.jp_sparse_pack(p, None, 3, 10, 0, 10, -1, 2, p, 10, cnt, p, 4096, None) == _abi.JP_ERR_ARG
+    assert lib.jp_sparse_pack(p, None, 4, 10, 5, 11, -1, 2, p, 10, cnt, p, 4096, None) == _abi.JP_ERR_ARG
+    assert lib.jp_sparse_pack(p, None, 4, 10, 0, 10, -1, 0, p, 10, cnt, p, 4096, None) == _abi.JP_ERR_ARG
+    assert lib.jp_sparse_pack(p, None, 4, 10, 0, 10, -1, 2, p, 10, cnt, p, 0, None) == _abi.JP_ERR_WORKSPACE
+    assert lib.jp_sparse_pack(p, None, 4, 1 << 31, 0, 10, -1, 2, p, 10, cnt, p, 4096, None) == _abi.JP_ERR_ARG
+    assert lib.jp_sparse_reduce_max(p, None, 8, 10, p, -1, None) == _abi.JP_ERR_ARG
+    assert lib.jp_sparse_gather(None, None, 4, 10, p, 3, None) == _abi.JP_ERR_ARG
+    assert lib.jp_sparse_scatter(p, None, 4, 10, None, 3, None) == _abi.JP_ERR_ARG
+    assert lib.jp_sparse_scratch_bytes(1 << 24, 8) >= 8 * (2 * ((1 << 24) // 4096) + 8)
+    assert lib.jp_sparse_scratch_bytes(-1, 8) == 0
 
 
 def test_bad_arguments():

@@ -28,7 +28,7 @@ def _free_port():
     return p
 
 
-def _worker(rank, world, port, case, q):
+def _worker(rank, world, port, case, q, exchange="dense"):
     sys.path[:0] = [ROOT, os.path.join(ROOT, "tests")]
     os.environ.update(MASTER_ADDR="127.0.0.1", MASTER_PORT=str(port))
     dist.init_process_group("gloo", rank=rank, world_size=world)
@@ -38,11 +38,12 @@ def _worker(rank, world, port, case, q):
         import paper_conf_icpp_hanzlw13_b200 as jp
         from paper_conf_icpp_hanzlw13_b200 import dist as jd
         import synth
-        from helpers import to_oracle
+        from helpers import region_workload, to_oracle
 
         wl = {"c1_0": lambda: synth.config1(0.0, n=600), "c1_5": lambda: synth.config1(0.05, n=600),
               "c4": lambda: synth.config4(n=700, slots=64), "c3": lambda: synth.config3(0.02, n=512),
-              "c2": lambda: synth.config2(n=901)}[case]()
+              "c2": lambda: synth.config2(n=901), "c5tail": lambda: region_workload(synth.config5(n=1 << 11), 3 << 9, 1 << 11),
+              "c5head": lambda: region_workload(synth.config5(n=1 << 11), 0, 1 << 10)}[case]()
         ref = to_oracle(wl)
         _, A_exp, T_exp = O.run_seq(ref)
         p_exp = O.profile(ref)
@@ -57,7 +58,8 @@ def _worker(rank, world, port, case, q):
             return
         loop = full.range(b, e)
         ws = torch.zeros(jp.jp_workspace_bytes(loop), dtype=torch.uint8)
-        res = jd.schedule_partitioned(loop, ws, full_loop=full, engine=fe)
+        jd.OWNER_MIN_LEN = 0   # small test tables still take the owner form
+        res = jd.schedule_partitioned(loop, ws, full_loop=full, engine=fe, exchange=exchange)
         prof_ok = (res["prof"]["raw_iters"], res["prof"]["war_iters"], res["prof"]["waw_iters"],
                    res["prof"]["first_raw_iter"]) == (p_exp["raw_iters"], p_exp["war_iters"], p_exp["waw_iters"],
                                                       p_exp["first_raw_iter"])
@@ -72,11 +74,11 @@ def _worker(rank, world, port, case, q):
         dist.destroy_process_group()
 
 
-def run_world(world, case):
+def run_world(world, case, exchange="dense"):
     ctx = mp.get_context("spawn")
     q = ctx.Queue()
     port = _free_port()
-    ps = [ctx.Process(target=_worker, args=(r, world, port, case, q)) for r in range(world)]
+    ps = [ctx.Process(target=_worker, args=(r, world, port, case, q, exchange)) for r in range(world)]
     for p in ps:
         p.start()
     out = [q.get(timeout=300) for _ in range(world)]
@@ -85,11 +87,13 @@ def run_world(world, case):
     return sorted(out)
 
 
+@pytest.mark.parametrize("exchange", ["dense", "owner"])
 @pytest.mark.parametrize("world", [2, 3])
 @pytest.mark.parametrize("case,mode", [("c1_0", "DOALL"), ("c1_5", "TLS"), ("c4", "PRIVATIZED"),
-                                       ("c3", "TLS"), ("c2", None)])
-def test_partitioned_schedule_matches_oracle(world, case, mode):
-    out = run_world(world, case)
+                                       ("c3", "TLS"), ("c2", None), ("c5tail", "PRIVATIZED"),
+                                       ("c5head", "DOALL")])
+def test_partitioned_schedule_matches_oracle(world, case, mode, exchange):
+    out = run_world(world, case, exchange)
     assert [o[1] for o in out] == [True] * world, out
     if mode:
         assert all(o[2] == mode for o in out), out

@@ -23,7 +23,7 @@ def _port():
     return p
 
 
-def _worker(rank, world, port, case, q):
+def _worker(rank, world, port, case, q, exchange="dense"):
     sys.path[:0] = [ROOT, os.path.join(ROOT, "tests")]
     os.environ.update(MASTER_ADDR="127.0.0.1", MASTER_PORT=str(port))
     dist.init_process_group("gloo", rank=rank, world_size=world)
@@ -32,11 +32,13 @@ def _worker(rank, world, port, case, q):
         import paper_conf_icpp_hanzlw13_b200 as jp
         from paper_conf_icpp_hanzlw13_b200 import dist as jd
         import synth
-        from helpers import to_oracle
+        from helpers import region_workload, to_oracle
         dev = torch.device("cuda:0")
         wl = {"c1_0": lambda: synth.config1(0.0), "c1_5": lambda: synth.config1(0.05),
               "c4": lambda: synth.config4(n=(1 << 18) + 5), "c3": lambda: synth.config3(0.01, n=1 << 16),
-              "c5tail": lambda: synth.config5(n=1 << 14)}[case]()
+              "c5tail": lambda: synth.config5(n=1 << 14),
+              "c5priv": lambda: region_workload(synth.config5(n=1 << 18), 3 << 16, 1 << 18),
+              "c5head": lambda: region_workload(synth.config5(n=1 << 18), 0, 1 << 17)}[case]()
         ref = to_oracle(wl)
         _, A_exp, T_exp = O.run_seq(ref)
         g = wl.to(dev)
@@ -44,7 +46,8 @@ def _worker(rank, world, port, case, q):
         b, e = jd.sharing_ranges(wl.n, world)[rank]
         loop = full.range(b, e)
         ws = jp.workspace(loop)
-        res = jd.schedule_partitioned(loop, ws, full_loop=full)
+        jd.OWNER_MIN_LEN = 1 << 12
+        res = jd.schedule_partitioned(loop, ws, full_loop=full, exchange=exchange)
         torch.cuda.synchronize()
         if wl.op == O.OP_PRIV_TMP:
             ok = g.A.cpu().numpy()[b:e].tobytes() == A_exp[b:e].tobytes() and \
@@ -61,13 +64,14 @@ def _worker(rank, world, port, case, q):
         dist.destroy_process_group()
 
 
+@pytest.mark.parametrize("exchange", ["dense", "owner"])
 @pytest.mark.parametrize("case,mode", [("c1_0", "DOALL"), ("c1_5", "TLS"), ("c4", "PRIVATIZED"), ("c3", "TLS"),
-                                       ("c5tail", "TLS")])
-def test_two_ranks_one_gpu(case, mode):
+                                       ("c5tail", "TLS"), ("c5priv", "PRIVATIZED"), ("c5head", "DOALL")])
+def test_two_ranks_one_gpu(case, mode, exchange):
     ctx = mp.get_context("spawn")
     q = ctx.Queue()
     port = _port()
-    ps = [ctx.Process(target=_worker, args=(r, 2, port, case, q)) for r in range(2)]
+    ps = [ctx.Process(target=_worker, args=(r, 2, port, case, q, exchange)) for r in range(2)]
     for p in ps:
         p.start()
     out = sorted(q.get(timeout=600) for _ in range(2))
