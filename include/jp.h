@@ -367,6 +367,38 @@ jp_status jp_schedule_workflow(const jp_loop *loops /* host [n] */, int32_t n, c
 /* Apply packed last-writer keys: arr[a] = keys[a] ? lo32(keys[a]) : arr[a]. */
 jp_status jp_merge_apply(void *arr, int64_t len, const int64_t *keys, jp_stream_t st);
 
+/* ---- task sharing with cross-boundary spill --------
+ * the part of the iteration space before the boundary "is divided
+ * into uniform chunks of moderate size, which are executed ... in an ascending
+ * order, while the right part is executed ... in a descending order"; the two
+ * consumers meet wherever the faster one gets to.  Generalised to k ranks:
+ * rank k's range (its task-sharing share, jp_plan_sharing) is cut into
+ * ceil(n_k / chunk) chunks; rank k consumes its own chunks ascending and, once
+ * they are all claimed, takes chunks DESCENDING from the tail of the rank with
+ * the most unclaimed chunks (ties: lowest rank; reading A18).
+ *
+ * views (host [world], world <= 8): every rank's shard as a loop descriptor
+ * whose pointers are valid in THIS process (the caller maps peer shards, e.g.
+ * with jp_ipc_import; on one device they are plain pointers).  Affine shards
+ * only: all index arrays NULL, ident_off 0, the same op / dtype / c0 / c1.
+ * ctr (device [world] uint64, visible to every rank, zero before ANY rank
+ * starts): ctr[k] = (tail claims << 32) | head claims of rank k's chunks,
+ * advanced with one system-scope atomicAdd per claim, so every chunk runs
+ * exactly once whatever the interleaving.  stats (device [3] int64, nullable,
+ * accumulated: the caller zeroes): iterations of own chunks, iterations
+ * stolen, chunks stolen by this executor.  max_ctas > 0 caps the grid.
+ * Results are complete when EVERY rank's launch has finished (the caller
+ * synchronises and barriers).  Stream-ordered.                               */
+jp_status jp_run_doall_spill(const jp_loop *views /* host [world] */, int32_t world, int32_t me, int64_t chunk,
+                             unsigned long long *ctr, int64_t *stats, int32_t max_ctas, jp_stream_t st);
+/* CUDA IPC plumbing for the spill (peer shards and the counter table):
+ * export: a 64-byte handle (host) of the allocation holding ptr, and ptr's
+ * byte offset in it; import (in another process): *ptr = mapped base + offset
+ * (peer access enabled lazily); close: unmap what import returned.           */
+jp_status jp_ipc_export(const void *ptr, void *handle /* host, 64 B */, int64_t *offset /* host */);
+jp_status jp_ipc_import(const void *handle /* host, 64 B */, int64_t offset, void **ptr /* host */);
+jp_status jp_ipc_close(void *ptr, int64_t offset);
+
 /* ---- owner-partitioned sparse exchange --------
  * Building blocks for the "one exchange step" of partitioned loops with
  * indirect writes: the whole-loop first-writer / first-reader tables of the

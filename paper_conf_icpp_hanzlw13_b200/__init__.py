@@ -25,6 +25,7 @@ __all__ = [
     "jp_profile_classify", "jp_profile_density", "jp_select_mode", "jp_run_doall", "jp_run_privatized",
     "jp_priv_stream", "jp_priv_finalize", "jp_doall_kernel", "jp_tls_guide", "tls_first_window", "jp_run_tls", "jp_schedule", "jp_stage_bytes", "jp_schedule_host",
     "jp_plan_sharing", "jp_plan_stealing", "jp_merge_apply",
+    "jp_run_doall_spill", "jp_ipc_export", "jp_ipc_import", "jp_ipc_close",
     "jp_sparse_scratch_bytes", "jp_sparse_pack", "jp_sparse_reduce_max", "jp_sparse_gather", "jp_sparse_scatter",
     "jp_last_error", "jp_version", "jp_launch_count",
 ]
@@ -330,6 +331,34 @@ def jp_plan_stealing(tasks, world: int, chunk_iters: int, speed=None, speed_tls:
 
 def jp_merge_apply(arr: torch.Tensor, keys: torch.Tensor, stream=None):
     check(lib().jp_merge_apply(arr.data_ptr(), arr.numel(), keys.data_ptr(), _stream(stream)))
+
+
+# ---- task sharing with cross-boundary spill (jp.h, M1 / C8) --------------
+def jp_run_doall_spill(views, me: int, chunk: int, ctr: torch.Tensor, stats=None, max_ctas: int = 0, stream=None):
+    """views: every rank's affine shard (Loop or jp_loop with pointers valid here);
+    ctr: int64 [world] device counters, zero before any rank starts; stats:
+    int64 [3] device accumulator (own iters, stolen iters, stolen chunks)."""
+    cs = [v.c if isinstance(v, Loop) else v for v in views]
+    arr = (_abi.jp_loop * len(cs))(*cs)
+    check(lib().jp_run_doall_spill(arr, len(cs), int(me), int(chunk), ctr.data_ptr(), _ptr(stats), int(max_ctas),
+                                   _stream(stream)))
+
+
+def jp_ipc_export(t: torch.Tensor) -> tuple[bytes, int]:
+    h = C.create_string_buffer(64)
+    off = C.c_int64()
+    check(lib().jp_ipc_export(t.data_ptr(), h, C.byref(off)))
+    return h.raw, off.value
+
+
+def jp_ipc_import(handle: bytes, offset: int) -> int:
+    p = C.c_void_p()
+    check(lib().jp_ipc_import(C.create_string_buffer(handle, 64), int(offset), C.byref(p)))
+    return int(p.value)
+
+
+def jp_ipc_close(ptr: int, offset: int):
+    check(lib().jp_ipc_close(C.c_void_p(ptr), int(offset)))
 
 
 # ---- owner-partitioned sparse exchange (jp.h, NEXT-2) ----------------------

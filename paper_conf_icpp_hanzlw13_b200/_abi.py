@@ -111,6 +111,10 @@ SIGNATURES = [
     ("jp_schedule_workflow", _I32, [_P(jp_loop), _I32, _P(jp_sched_cfg), _P(_V), _P(_SZ), _P(jp_sched_result),
                                     _P(jp_workflow_plan), _V]),
     ("jp_merge_apply", _I32, [_V, _I64, _V, _V]),
+    ("jp_run_doall_spill", _I32, [_P(jp_loop), _I32, _I32, _I64, _V, _V, _I32, _V]),
+    ("jp_ipc_export", _I32, [_V, _V, _P(_I64)]),
+    ("jp_ipc_import", _I32, [_V, _I64, _P(_V)]),
+    ("jp_ipc_close", _I32, [_V, _I64]),
     ("jp_sparse_scratch_bytes", _SZ, [_I64, _I32]),
     ("jp_sparse_pack", _I32, [_V, _V, _I32, _I64, _I64, _I64, _I64, _I32, _V, _I64, _P(_I64), _V, _SZ, _V]),
     ("jp_sparse_reduce_max", _I32, [_V, _V, _I32, _I64, _V, _I64, _V]),

@@ -655,6 +655,77 @@ jp_status jp_merge_apply(void *arr, int64_t len, const int64_t *keys, jp_stream_
 }
 
 // ---------------------------------------------------------------------------
+// task sharing with cross-boundary spill (M1, C8) and the IPC plumbing it needs
+// ---------------------------------------------------------------------------
+jp_status jp_run_doall_spill(const jp_loop *views, int32_t world, int32_t me, int64_t chunk,
+                             unsigned long long *ctr, int64_t *stats, int32_t max_ctas, jp_stream_t st) {
+  if (!views || world < 1 || world > kSpillRanks || me < 0 || me >= world)
+    return fail(JP_ERR_ARG, "need 1 <= world <= %d and 0 <= me < world", kSpillRanks);
+  if (chunk < 1 || !ctr) return fail(JP_ERR_ARG, "need chunk >= 1 and a counter table");
+  Job jobs[kSpillRanks];
+  for (int k = 0; k < world; k++) {
+    const jp_loop *L = &views[k];
+    JP_TRY(check_loop(L));
+    if (L->r || L->r2 || L->w || L->s || L->ident_off != 0)
+      return fail(JP_ERR_UNSUPPORTED, "spill runs affine shards only (NULL index arrays, ident_off 0)");
+    if (L->op != views[0].op || L->dtype != views[0].dtype || L->c0.i != views[0].c0.i || L->c1.i != views[0].c1.i)
+      return fail(JP_ERR_ARG, "every rank's view must run the same body");
+    if ((L->n + chunk - 1) / chunk >= (1LL << 31)) return fail(JP_ERR_ARG, "too many chunks");
+    jobs[k] = make_job(L);
+  }
+  JP_TRY(need_device());
+  JP_CUDA(launch_doall_spill(jobs, world, me, chunk, ctr, stats, max_ctas, (cudaStream_t)st), "doall spill");
+  return JP_OK;
+}
+
+typedef int (*cu_range_fn)(unsigned long long *, size_t *, unsigned long long);
+static cu_range_fn cu_mem_range() {
+  static cu_range_fn fn = nullptr;
+  static std::once_flag once;
+  std::call_once(once, [] {
+    void *p = nullptr;
+    cudaDriverEntryPointQueryResult q;
+    if (cudaGetDriverEntryPoint("cuMemGetAddressRange", &p, cudaEnableDefault, &q) == cudaSuccess &&
+        q == cudaDriverEntryPointSuccess)
+      fn = reinterpret_cast<cu_range_fn>(p);
+  });
+  return fn;
+}
+
+jp_status jp_ipc_export(const void *ptr, void *handle, int64_t *offset) {
+  if (!ptr || !handle || !offset) return fail(JP_ERR_ARG, "NULL argument");
+  JP_TRY(need_device());
+  cu_range_fn fn = cu_mem_range();
+  unsigned long long base = 0;
+  size_t size = 0;
+  if (!fn || fn(&base, &size, (unsigned long long)(uintptr_t)ptr) != 0)
+    return fail(JP_ERR_CUDA, "cuMemGetAddressRange failed for %p", ptr);
+  cudaIpcMemHandle_t h;
+  JP_CUDA(cudaIpcGetMemHandle(&h, (void *)(uintptr_t)base), "cudaIpcGetMemHandle");
+  memcpy(handle, &h, sizeof h);
+  *offset = (int64_t)((uintptr_t)ptr - base);
+  return JP_OK;
+}
+
+jp_status jp_ipc_import(const void *handle, int64_t offset, void **ptr) {
+  if (!handle || !ptr || offset < 0) return fail(JP_ERR_ARG, "bad IPC import arguments");
+  JP_TRY(need_device());
+  cudaIpcMemHandle_t h;
+  memcpy(&h, handle, sizeof h);
+  void *base = nullptr;
+  JP_CUDA(cudaIpcOpenMemHandle(&base, h, cudaIpcMemLazyEnablePeerAccess), "cudaIpcOpenMemHandle");
+  *ptr = static_cast<char *>(base) + offset;
+  return JP_OK;
+}
+
+jp_status jp_ipc_close(void *ptr, int64_t offset) {
+  if (!ptr || offset < 0) return fail(JP_ERR_ARG, "bad IPC close arguments");
+  JP_TRY(need_device());
+  JP_CUDA(cudaIpcCloseMemHandle(static_cast<char *>(ptr) - offset), "cudaIpcCloseMemHandle");
+  return JP_OK;
+}
+
+// ---------------------------------------------------------------------------
 // owner-partitioned sparse exchange (NEXT-2)
 // ---------------------------------------------------------------------------
 static jp_status check_sparse(const void *t0, int32_t elem, int64_t len, const void *rows, int64_t m) {

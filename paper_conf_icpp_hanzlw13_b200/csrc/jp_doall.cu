@@ -11,6 +11,7 @@
 //   coalesced index streams, gathered/scattered element accesses.
 #include <atomic>
 #include <cstdlib>
+#include <cstring>
 #include "jp_host.h"
 
 namespace jp {
@@ -160,7 +161,7 @@ __global__ void __launch_bounds__(256) k_doall_generic(DLoop L) {
   }
 }
 
-static bool aligned16(const void *p) { return ((uintptr_t)p & 15) == 0; }
+__host__ __device__ static inline bool aligned16(const void *p) { return ((uintptr_t)p & 15) == 0; }
 
 // affine DOALL kernel choice (jp_doall_kernel): 0 LDG/STG.128 grid-stride, 1 bulk-copy (TMA) staged
 // (default: config 2 measured 6.48 vs 6.25 TB/s)
@@ -203,6 +204,151 @@ static void run_doall(const DLoop &d, cudaStream_t st, int max_ctas) {
     k_doall_generic<OP, DT><<<grid, 256, 0, st>>>(d);
   }
   note_launch();
+}
+
+// ---------------------------------------------------------------------------
+// k_doall_spill: task sharing with cross-boundary spill (M1; C8).
+// Every rank's range is cut into uniform chunks.  Rank k's chunk counter
+// ctr[k] packs (tail claims << 32 | head claims); one system-scope 64-bit
+// atomicAdd claims a chunk and sees both counts at once, so a chunk c is taken
+// exactly once: the owner claims ascending (head h valid iff h + t < nch),
+// an idle rank claims descending from the tail (chunk nch-1-t, same test).
+// Once its own range is exhausted a CTA steals from the rank with the most
+// unclaimed chunks, ties to the lowest rank (reading A18).  The views are the
+// ranks' shards with pointers valid in this process (peer memory mapped over
+// NVLink through CUDA IPC on a multi-GPU node), so a stolen chunk is read and
+// written where it lives.
+// ---------------------------------------------------------------------------
+constexpr int kSpillMaxRanks = 8;
+struct SpillArgs {
+  DLoop v[kSpillMaxRanks];
+  int64_t nch[kSpillMaxRanks];
+  unsigned long long *ctr;
+  int64_t *stats;   // [0] own iterations, [1] stolen iterations, [2] stolen chunks (this executor)
+  int64_t chunk;
+  int world, me;
+};
+
+__device__ __forceinline__ bool spill_claim(unsigned long long *ctr, int64_t nch, bool tail, int64_t &c) {
+  const unsigned long long old = atomicAdd_system(ctr, tail ? (1ull << 32) : 1ull);
+  const int64_t h = (uint32_t)old, t = (uint32_t)(old >> 32);
+  if (h + t >= nch) return false;
+  c = tail ? nch - 1 - t : h;
+  return true;
+}
+
+template <int OP, int DT>
+__device__ __forceinline__ void spill_chunk(const DLoop &L, int64_t s, int64_t e) {
+  constexpr bool readsA = OP != JP_OP_PRIV_TMP;
+  constexpr bool readsX = OP == JP_OP_SAXPY || OP == JP_OP_PRIV_TMP;
+  int64_t v_end = 0;
+  if (aligned16(L.A + s) && (!readsX || aligned16(L.X + s)) && (OP != JP_OP_PRIV_TMP || aligned16(L.T + s))) {
+    const int64_t nvec = (e - s) >> 2;
+    v_end = nvec << 2;
+    const uint4 *X4 = reinterpret_cast<const uint4 *>(L.X + s);
+    uint4 *A4 = reinterpret_cast<uint4 *>(L.A + s);
+    uint4 *T4 = reinterpret_cast<uint4 *>(L.T + s);
+    for (int64_t v0 = threadIdx.x; v0 < nvec; v0 += kAffThreads * kAffUnroll) {
+      uint4 a[kAffUnroll], x[kAffUnroll], t[kAffUnroll];
+#pragma unroll
+      for (int u = 0; u < kAffUnroll; u++) {
+        const int64_t v = v0 + (int64_t)u * kAffThreads;
+        if (v < nvec) {
+          if constexpr (readsA) a[u] = __ldcs(A4 + v);
+          if constexpr (readsX) x[u] = __ldcs(X4 + v);
+        }
+      }
+#pragma unroll
+      for (int u = 0; u < kAffUnroll; u++) {
+        const int64_t v = v0 + (int64_t)u * kAffThreads;
+        if (v < nvec) {
+          vec_body<OP, DT>(x[u], a[u], t[u], L.c0, L.c1);
+          __stcs(A4 + v, a[u]);
+          if constexpr (OP == JP_OP_PRIV_TMP) __stcs(T4 + v, t[u]);
+        }
+      }
+    }
+  }
+  for (int64_t i = s + v_end + threadIdx.x; i < e; i += kAffThreads) {
+    uint32_t va = 0, vt = 0;
+    body_values<OP, DT>(L, i, L.A, va, vt);
+    if constexpr (OP == JP_OP_PRIV_TMP) L.T[i] = vt;
+    L.A[i] = va;
+  }
+}
+
+template <int OP, int DT>
+__global__ void __launch_bounds__(kAffThreads) k_doall_spill(const __grid_constant__ SpillArgs P) {
+  __shared__ int s_rank;
+  __shared__ long long s_chunk;
+  int64_t own = 0, stolen = 0, nst = 0;
+  bool mine = true;
+  for (;;) {
+    if (threadIdx.x == 0) {
+      int rk = -1;
+      int64_t c = 0;
+      if (mine && spill_claim(&P.ctr[P.me], P.nch[P.me], false, c)) rk = P.me;
+      else mine = false;
+      while (rk < 0) {   // steal: the rank with the most unclaimed chunks, ties to the lowest
+        int best = -1;
+        int64_t most = 0;
+        for (int k = 0; k < P.world; k++) {
+          if (k == P.me) continue;
+          const unsigned long long v = *(volatile unsigned long long *)&P.ctr[k];
+          const int64_t left = P.nch[k] - (int64_t)(uint32_t)v - (int64_t)(uint32_t)(v >> 32);
+          if (left > most) { most = left; best = k; }
+        }
+        if (best < 0) break;
+        if (spill_claim(&P.ctr[best], P.nch[best], true, c)) rk = best;
+      }
+      s_rank = rk;
+      s_chunk = c;
+    }
+    __syncthreads();
+    const int rk = s_rank;
+    const int64_t c = s_chunk;
+    __syncthreads();
+    if (rk < 0) break;
+    const DLoop &L = P.v[rk];
+    const int64_t s = c * P.chunk, e = s + P.chunk < L.n ? s + P.chunk : L.n;
+    spill_chunk<OP, DT>(L, s, e);
+    if (threadIdx.x == 0) {
+      if (rk == P.me) own += e - s;
+      else { stolen += e - s; nst++; }
+    }
+  }
+  if (threadIdx.x == 0 && P.stats) {
+    if (own) atomicAdd(reinterpret_cast<unsigned long long *>(&P.stats[0]), (unsigned long long)own);
+    if (stolen) {
+      atomicAdd(reinterpret_cast<unsigned long long *>(&P.stats[1]), (unsigned long long)stolen);
+      atomicAdd(reinterpret_cast<unsigned long long *>(&P.stats[2]), (unsigned long long)nst);
+    }
+  }
+}
+
+template <int OP, int DT>
+static void run_spill(const SpillArgs &P, int grid, cudaStream_t st) {
+  k_doall_spill<OP, DT><<<grid, kAffThreads, 0, st>>>(P);
+  note_launch();
+}
+
+cudaError_t launch_doall_spill(const Job *views, int world, int me, int64_t chunk, unsigned long long *ctr,
+                               int64_t *stats, int max_ctas, cudaStream_t st) {
+  SpillArgs P;
+  memset(&P, 0, sizeof P);
+  for (int k = 0; k < world; k++) {
+    P.v[k] = views[k].d;
+    P.nch[k] = (views[k].d.n + chunk - 1) / chunk;
+  }
+  P.ctr = ctr;
+  P.stats = stats;
+  P.chunk = chunk;
+  P.world = world;
+  P.me = me;
+  int grid = num_sms() * 4;   // 256-thread CTAs, 4 per SM resident
+  if (max_ctas > 0 && grid > max_ctas) grid = max_ctas;
+  JP_DISPATCH(views[0].op, views[0].dt, run_spill, P, grid, st);
+  return launch_check();
 }
 
 cudaError_t launch_doall(const Job &j, cudaStream_t st, int max_ctas) {

@@ -62,6 +62,10 @@ cudaError_t launch_priv_stream(const Job &j, void *ws, const Layout &lo, bool cl
                                cudaStream_t st, int max_ctas = 0, bool fuse_apply = false, bool *applied = nullptr);
 cudaError_t launch_priv_finalize(const Job &j, void *ws, const Layout &lo, cudaStream_t st);
 cudaError_t launch_merge_apply(void *arr, int64_t len, const int64_t *keys, cudaStream_t st);
+// task sharing with cross-boundary spill (jp_doall.cu, C8): views[k] = rank k's affine shard
+constexpr int kSpillRanks = 8;
+cudaError_t launch_doall_spill(const Job *views, int world, int me, int64_t chunk, unsigned long long *ctr,
+                               int64_t *stats, int max_ctas, cudaStream_t st);
 // owner-partitioned sparse exchange (jp_exchange.cu)
 size_t sparse_scratch_bytes(int64_t len, int world);
 int64_t sparse_pack_tiles(int64_t len, int64_t lo, int64_t hi, int world);

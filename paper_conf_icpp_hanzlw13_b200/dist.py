@@ -221,6 +221,91 @@ def schedule_partitioned(loop, ws, group=None, tau_high: float = 0.25, tls_windo
     return res
 
 
+class SpillGroup:
+    """Task sharing with cross-boundary spill across the ranks (M1, P:L350-353;
+    C8): every rank maps every other rank's affine shard and rank 0's chunk
+    counter table through CUDA IPC once; ``run`` then executes the whole loop
+    with jp_run_doall_spill on every rank -- each rank consumes its own chunks
+    ascending and, when done, takes the most-loaded rank's chunks descending,
+    reading and writing them in the peer's memory over NVLink.  No collective
+    moves data; two barriers bracket the run (counters zero before any rank
+    starts; every chunk written before any rank reads its shard)."""
+
+    def __init__(self, shard, group=None):
+        import paper_conf_icpp_hanzlw13_b200 as jp
+        self.jp, self.group = jp, group
+        self.world, self.rank = world_rank(group)
+        if self.world > 8:
+            raise ValueError("spill supports up to 8 ranks (one node)")
+        self.shard = shard
+        dev = shard.tensors["A"].device
+        self.ctr = torch.zeros(self.world, dtype=torch.int64, device=dev)
+        self.stats = torch.zeros(3, dtype=torch.int64, device=dev)
+        self._opened = []
+        views = [shard.c]
+        if self.world > 1:
+            mine = {k: (None if shard.tensors[k] is None else jp.jp_ipc_export(shard.tensors[k])) for k in "AXT"}
+            mine["ctr"] = jp.jp_ipc_export(self.ctr) if self.rank == 0 else None
+            allinfo = [None] * self.world
+            dist.all_gather_object(allinfo, mine, group=group)
+            views = []
+            for k, info in enumerate(allinfo):
+                if k == self.rank:
+                    views.append(shard.c)
+                    continue
+                v = _abi.jp_loop.from_buffer_copy(shard.c)
+                for name in "AXT":
+                    if info[name] is not None:
+                        ptr = jp.jp_ipc_import(*info[name])
+                        self._opened.append((ptr, info[name][1]))
+                        setattr(v, name, ptr)
+                views.append(v)
+            if self.rank != 0:
+                ptr = jp.jp_ipc_import(*allinfo[0]["ctr"])
+                self._opened.append((ptr, allinfo[0]["ctr"][1]))
+                self._ctr_ptr = ptr
+            # every rank's shard has the same length semantics; n per rank from the peers
+            ns = [None] * self.world
+            dist.all_gather_object(ns, (shard.n, shard.c.len_A, shard.c.len_X, shard.c.len_T), group=group)
+            for k, v in enumerate(views):
+                v.n, v.len_A, v.len_X, v.len_T = ns[k]
+        self.views = views
+
+    def _ctr(self):
+        if self.rank == 0 or self.world == 1:
+            return self.ctr
+        return _RawPtr(self._ctr_ptr)
+
+    def run(self, chunk: int = 1 << 20, max_ctas: int = 0, stream=None) -> dict:
+        if self.rank == 0:
+            self.ctr.zero_()
+        self.stats.zero_()
+        if self.world > 1:
+            torch.cuda.synchronize()
+            dist.barrier(group=self.group)
+        self.jp.jp_run_doall_spill(self.views, self.rank, chunk, self._ctr(), self.stats, max_ctas, stream)
+        if self.world > 1:
+            torch.cuda.synchronize()
+            dist.barrier(group=self.group)
+        own, stolen, nst = (int(x) for x in self.stats.tolist())
+        return {"own_iters": own, "stolen_iters": stolen, "stolen_chunks": nst}
+
+    def close(self):
+        for ptr, off in self._opened:
+            self.jp.jp_ipc_close(ptr, off)
+        self._opened = []
+
+
+class _RawPtr:
+    """A device pointer posing as a tensor for the binding (data_ptr only)."""
+
+    def __init__(self, ptr):
+        self.ptr = ptr
+
+    def data_ptr(self):
+        return self.ptr
+
+
 def stealing_plan(tasks, world: int, chunk_iters: int, speed=None, speed_tls: float = 0.05, engine=None):
     """Alg. 1 as a deterministic plan: [(start, end, mode, owner)] and #stolen."""
     return _engine(engine).jp_plan_stealing(tasks, world, chunk_iters, speed, speed_tls)

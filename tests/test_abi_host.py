@@ -177,6 +177,10 @@ def test_compute_calls_fail_loudly_without_gpu():
     with pytest.raises(jp.JPError) as e:
         jp.jp_schedule(L, torch.zeros(1 << 20, dtype=torch.uint8))
     assert e.value.status == _abi.JP_ERR_CUDA
+    Y = torch.zeros(64, dtype=torch.float32)
+    with pytest.raises(jp.JPError) as e:
+        jp.jp_run_doall_spill([jp.Loop(1, 1, 64, Y, X=Y.clone(), c0=2.0)], 0, 16, torch.zeros(1, dtype=torch.int64))
+    assert e.value.status == _abi.JP_ERR_CUDA
     t = torch.zeros(100, dtype=torch.int32)
     with pytest.raises(jp.JPError) as e:
         jp.jp_sparse_pack(t, None, -1, 2)
