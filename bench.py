@@ -391,6 +391,131 @@ def partitioned_config4(jp, dev, st, world, rank, steps):
             "profile_ms": prof_ms, "collective": "torch.distributed all_reduce MAX (C4, 8 KiB int64)"}
 
 
+def partitioned_spill(jp, dev, st, world, rank, steps):
+    """Config 2 under task sharing with cross-boundary spill (M1, C8): every rank
+    runs jp_run_doall_spill over its shard and steals chunks (2^16 iterations,
+    reading A17) descending from the most-loaded peer's shard over CUDA IPC.
+    Step = counter reset + barrier + kernel + barrier; max over ranks.  At N = 1
+    also a two-virtual-rank imbalance on one GPU: the second "rank" capped to 8
+    CTAs (a slow device), static sharing vs spill, wall clock around both
+    streams."""
+    import synth
+    from paper_conf_icpp_hanzlw13_b200 import dist as jd
+    s0, s1 = jp.jp_plan_sharing(N2, world)[rank]
+    wl = synth.config2(n=N2, device=dev, start=s0, count=s1 - s0)
+    L = jp.Loop.from_workload(wl, iter_base=s0)
+    sg = jd.SpillGroup(L)
+    for _ in range(3):
+        sg.run()
+    kernel_ms = None
+    if world == 1:   # the spill kernel alone (CUDA events on the launching stream)
+        ctr = torch.zeros(1, dtype=torch.int64, device=dev)
+        evs = []
+        for _ in range(steps):
+            ctr.zero_()
+            a, z = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            a.record(st)
+            jp.jp_run_doall_spill([L], 0, 1 << 16, ctr, None, 0, st)
+            z.record(st)
+            evs.append((a, z))
+        torch.cuda.synchronize()
+        kernel_ms = statistics.median([a.elapsed_time(z) for a, z in evs])
+    ts, res = [], None
+    for _ in range(steps):
+        torch.cuda.synchronize()
+        t0 = time.perf_counter()
+        res = sg.run()
+        ts.append(time.perf_counter() - t0)
+    ms = max_over_ranks(statistics.median(ts) * 1e3, world, dev)
+    sg.close()
+    out = {"workload": "config2 SAXPY fp32 N=2^28, task sharing + spill (chunk 2^16)", "ms": ms,
+           "iters_per_s": N2 / (ms * 1e-3), "rank0": res, "timing": "wall clock incl. 2 barriers, max over ranks"}
+    if kernel_ms:
+        out["kernel_ms"] = kernel_ms
+        out["kernel_GBps"] = BYTES_PER_ITER_SAXPY * N2 / (kernel_ms * 1e-3) / 1e9
+    del wl, L, sg
+    if world == 1:
+        hbm, _ = peaks()
+        half = N2 // 2
+        shards = [synth.config2(n=N2, device=dev, start=k * half, count=half) for k in range(2)]
+        Ls = [jp.Loop.from_workload(x, iter_base=k * half) for k, x in enumerate(shards)]
+        sts = [torch.cuda.Stream(), torch.cuda.Stream()]
+        ctr = torch.zeros(2, dtype=torch.int64, device=dev)
+        stats = torch.zeros(3, dtype=torch.int64, device=dev)
+
+        def once(spill):
+            ctr.zero_()
+            stats.zero_()
+            torch.cuda.synchronize()
+            t0 = time.perf_counter()
+            for k in range(2):
+                views = Ls if spill else [Ls[k]]
+                jp.jp_run_doall_spill(views, k if spill else 0, 1 << 16, ctr if spill else ctr[k:k + 1],
+                                      stats if k == 0 else None, 0 if k == 0 else 8, sts[k])
+            torch.cuda.synchronize()
+            return time.perf_counter() - t0
+
+        row = {}
+        for name, spill in (("static", False), ("spill", True)):
+            for _ in range(2):
+                once(spill)
+            t = statistics.median([once(spill) for _ in range(5)])
+            row[name] = {"ms": t * 1e3, "iters_per_s": N2 / t, "GBps": BYTES_PER_ITER_SAXPY * N2 / t / 1e9}
+            if spill:
+                own, stolen, nst = (int(x) for x in stats.tolist())
+                row[name].update({"fast_rank_own_iters": own, "fast_rank_stolen_iters": stolen})
+        row["note"] = "2 virtual ranks on one GPU (separate shards, streams); rank 1 capped to 8 CTAs"
+        out["imbalanced_2x1gpu"] = row
+        del shards, Ls
+    return out
+
+
+def exchange_cost(jp, dev, st):
+    """NEXT-2 on one GPU: rank 0 of 8 of config 3 (d = 1%) and config 5's
+    privatized tail: what the owner form sends vs the dense all_reduce, and the
+    time of its local kernels (pack, reduce, gather, scatter).  The all_to_all
+    itself needs several GPUs (unmeasured here)."""
+    import synth
+    from paper_conf_icpp_hanzlw13_b200 import dist as jd
+    out = {}
+    world = 8
+    wl = synth.config3(0.01, device=dev)
+    full = jp.Loop.from_workload(wl)
+    b, e = jd.sharing_ranges(wl.n, world)[0]
+    loop = full.range(b, e)
+    ws = jp.workspace(loop)
+    jp.jp_profile_stamp(loop, ws)
+    W = jd._region(ws, loop, "minW_A", torch.int32, jp)
+    R = jd._region(ws, loop, "minR_A", torch.int32, jp)
+
+    def ev(fn, k=5):
+        fn()
+        a, z = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        torch.cuda.synchronize()
+        a.record(st)
+        for _ in range(k):
+            fn()
+        z.record(st)
+        torch.cuda.synchronize()
+        return a.elapsed_time(z) / k
+
+    rows, counts = jp.jp_sparse_pack(W, R, -1, world)
+    pack_ms = ev(lambda: jp.jp_sparse_pack(W, R, -1, world))
+    R2 = rows.clone()
+    red_ms = ev(lambda: jp.jp_sparse_reduce_max(W, R, R2))
+    gat_ms = ev(lambda: jp.jp_sparse_gather(W, R, R2))
+    sca_ms = ev(lambda: jp.jp_sparse_scatter(W, R, R2))
+    dense = 2 * W.numel() * 4
+    out["config3_profile_C1"] = {
+        "rank_range": e - b, "rows": int(rows.shape[0]), "rows_per_owner": counts,
+        "owner_bytes_sent_per_rank": 2 * rows.numel() * 4, "dense_table_bytes": dense,
+        "dense_allreduce_bytes_sent_per_rank_ring": 2 * (world - 1) / world * dense,
+        "pack_ms": pack_ms, "reduce_ms": red_ms, "gather_ms": gat_ms, "scatter_ms": sca_ms}
+    del wl, full, loop, ws, W, R, rows, R2
+    torch.cuda.empty_cache()
+    return out
+
+
 def run_jp(args):
     import paper_conf_icpp_hanzlw13_b200 as jp
     import synth
@@ -479,10 +604,13 @@ def run_jp(args):
         torch.cuda.empty_cache()
         part = partitioned_config4(jp, dev, st, world, rank, 5)
         torch.cuda.empty_cache()
+        spill = partitioned_spill(jp, dev, st, world, rank, 5)
+        torch.cuda.empty_cache()
         if rank == 0:
-            out["partitioned"] = {"config4": part}
+            out["partitioned"] = {"config4": part, "config2_spill": spill}
         if world == 1:
             out["modes"] = modes_sweep(jp, dev, st)
+            out["modes"]["exchange_owner"] = exchange_cost(jp, dev, st)
     if rank == 0:
         out["cpu_baseline"] = oracle_baseline(1 << 25)
         print(json.dumps(out), flush=True)

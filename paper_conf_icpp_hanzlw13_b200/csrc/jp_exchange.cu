@@ -38,37 +38,39 @@ struct XTiles {
   }
 };
 
+// Warp w of a tile owns the kXPer * 32 consecutive entries starting at
+// b + w * kXPer * 32; round q reads entry (q, lane) = base + q * 32 + lane
+// (coalesced).  Returns the warp's ballots packed as per-lane flag bits
+// (bit q = flag of entry (q, lane)) and the warp's total.
 template <typename E, int NT>
-__device__ __forceinline__ bool x_full(const E *t0, const E *t1, int64_t a, E empty) {
-  if (t0[a] != empty) return true;
-  if constexpr (NT == 2) return t1[a] != empty;
-  return false;
-}
-
-// per thread: the flags of its kXPer consecutive entries of tile t
-template <typename E, int NT>
-__device__ __forceinline__ uint32_t x_flags(const E *t0, const E *t1, E empty, int64_t b, int64_t e) {
+__device__ __forceinline__ uint32_t x_flags(const E *t0, const E *t1, E empty, int64_t b, int64_t e, int &wtot) {
+  const int lane = threadIdx.x & 31, wid = threadIdx.x >> 5;
+  const int64_t a0 = b + (int64_t)wid * kXPer * 32 + lane;
   uint32_t f = 0;
-  const int64_t a0 = b + (int64_t)threadIdx.x * kXPer;
+  E v0[kXPer], v1[kXPer];
+#pragma unroll
+  for (int q = 0; q < kXPer; q++) {   // all loads first (16 in flight per lane)
+    const int64_t a = a0 + q * 32;
+    v0[q] = a < e ? t0[a] : empty;
+    if constexpr (NT == 2) v1[q] = a < e ? t1[a] : empty;
+  }
+  int tot = 0;
 #pragma unroll
   for (int q = 0; q < kXPer; q++) {
-    const int64_t a = a0 + q;
-    if (a < e && x_full<E, NT>(t0, t1, a, empty)) f |= 1u << q;
+    bool full = v0[q] != empty;
+    if constexpr (NT == 2) full = full || v1[q] != empty;
+    f |= (uint32_t)full << q;
+    tot += __popc(__ballot_sync(0xffffffffu, full));
   }
+  wtot = tot;
   return f;
 }
 
-// block-wide exclusive scan of v (kXThreads threads); *total = sum
-__device__ __forceinline__ int x_scan(int v, int *total) {
+// exclusive prefix of the warps' totals (one value per warp); *total = sum
+__device__ __forceinline__ int x_warp_scan(int wtot, int *total) {
   __shared__ int ws[kXThreads / 32];
   const int lane = threadIdx.x & 31, wid = threadIdx.x >> 5;
-  int x = v;
-#pragma unroll
-  for (int d = 1; d < 32; d <<= 1) {
-    const int y = __shfl_up_sync(0xffffffffu, x, d);
-    if (lane >= d) x += y;
-  }
-  if (lane == 31) ws[wid] = x;
+  if (lane == 0) ws[wid] = wtot;
   __syncthreads();
   int pre = 0, tot = 0;
 #pragma unroll
@@ -77,17 +79,17 @@ __device__ __forceinline__ int x_scan(int v, int *total) {
     if (w < wid) pre += s;
     tot += s;
   }
-  __syncthreads();
   *total = tot;
-  return pre + x - v;
+  return pre;
 }
 
 template <typename E, int NT>
 __global__ void __launch_bounds__(kXThreads) k_x_count(const E *t0, const E *t1, E empty, XTiles X, int64_t *cnt) {
   int64_t b, e;
   X.range(blockIdx.x, b, e);
-  int tot;
-  x_scan(__popc(x_flags<E, NT>(t0, t1, empty, b, e)), &tot);
+  int wtot, tot;
+  x_flags<E, NT>(t0, t1, empty, b, e, wtot);
+  x_warp_scan(wtot, &tot);
   if (threadIdx.x == 0) cnt[blockIdx.x] = tot;
 }
 
@@ -122,17 +124,25 @@ __global__ void __launch_bounds__(kXThreads) k_x_emit(const E *t0, const E *t1, 
                                                       E *rows, int64_t cap) {
   int64_t b, e;
   X.range(blockIdx.x, b, e);
-  const uint32_t f = x_flags<E, NT>(t0, t1, empty, b, e);
-  int tot;
-  int64_t r = off[blockIdx.x] + x_scan(__popc(f), &tot);
-  const int64_t a0 = b + (int64_t)threadIdx.x * kXPer;
-  for (uint32_t g = f; g; g &= g - 1, r++) {
-    const int64_t a = a0 + __ffs(g) - 1;
-    if (r >= cap) break;
-    E *row = rows + r * (1 + NT);
-    row[0] = (E)a;
-    row[1] = t0[a];
-    if constexpr (NT == 2) row[2] = t1[a];
+  int wtot, tot;
+  const uint32_t f = x_flags<E, NT>(t0, t1, empty, b, e, wtot);
+  const int lane = threadIdx.x & 31, wid = threadIdx.x >> 5;
+  int64_t r = off[blockIdx.x] + x_warp_scan(wtot, &tot);
+  const int64_t a0 = b + (int64_t)wid * kXPer * 32 + lane;
+  const uint32_t lt = (1u << lane) - 1u;
+#pragma unroll
+  for (int q = 0; q < kXPer; q++) {
+    const bool full = (f >> q) & 1u;
+    const uint32_t bal = __ballot_sync(0xffffffffu, full);
+    const int64_t ri = r + __popc(bal & lt);
+    if (full && ri < cap) {
+      const int64_t a = a0 + q * 32;
+      E *row = rows + ri * (1 + NT);
+      row[0] = (E)a;
+      row[1] = t0[a];
+      if constexpr (NT == 2) row[2] = t1[a];
+    }
+    r += __popc(bal);
   }
 }
 

@@ -276,7 +276,7 @@ class SpillGroup:
             return self.ctr
         return _RawPtr(self._ctr_ptr)
 
-    def run(self, chunk: int = 1 << 20, max_ctas: int = 0, stream=None) -> dict:
+    def run(self, chunk: int = 1 << 16, max_ctas: int = 0, stream=None) -> dict:
         if self.rank == 0:
             self.ctr.zero_()
         self.stats.zero_()
