@@ -367,6 +367,30 @@ jp_status jp_schedule_workflow(const jp_loop *loops /* host [n] */, int32_t n, c
 /* Apply packed last-writer keys: arr[a] = keys[a] ? lo32(keys[a]) : arr[a]. */
 jp_status jp_merge_apply(void *arr, int64_t len, const int64_t *keys, jp_stream_t st);
 
+/* ---- task stealing across ranks (SURVEY §8(e) "Mixed", Alg. 1) ----
+ * The multi-rank stealing scheme (paper_conf_icpp_hanzlw13_b200/dist.py
+ * schedule_stealing) needs, on every rank, the same task list and PDG that
+ * jp_schedule(STEALING) builds on one device:
+ * jp_plan_tasks: chunk_counts (host [3 * ceil(n / chunk_iters)]: raw, war, waw
+ * iteration counts of every chunk of the WHOLE loop L, e.g. the sum over the
+ * ranks of jp_profile_classify's chunk counts) -> tasks = maximal runs of
+ * chunks of one Fig. 2(b) mode (reading A19; at most 64, smaller runs merged
+ * into the stronger mode), tasks (host [3 * 64]) = (start, end, mode) each,
+ * *n_tasks; conf (host [64]): bit t of conf[u] set iff tasks t and u touch a
+ * common address and at least one writes it (reading B2), computed over L's
+ * accesses on this device (workspace JP_WS_ALL of L).  chunk_iters >= 1024, a
+ * multiple of 32.  syncs.                                                   */
+jp_status jp_plan_tasks(const jp_loop *L, const int64_t *chunk_counts /* host */, int64_t chunk_iters, double tau_high,
+                        void *ws, size_t ws_bytes, int64_t *tasks /* host [192] */, int32_t *n_tasks /* host */,
+                        uint64_t *conf /* host [64] */, jp_stream_t st);
+/* Packed last-writer keys (regions keys_A / keys_T of ws, NOT cleared) of what
+ * loop L has already written in place: for every iteration i and every
+ * indirectly written element a, keys[a] = max(keys[a], (iter_base+i+1) << 32 |
+ * bits(current a)).  Used after a TLS task ran in place on its pinned rank so
+ * that the other replicas receive its writes through C4 like every privatized
+ * task's (reading A9: last writer wins).  Stream-ordered.                   */
+jp_status jp_export_keys(const jp_loop *L, void *ws, size_t ws_bytes, jp_stream_t st);
+
 /* ---- task sharing with cross-boundary spill --------
  * the part of the iteration space before the boundary "is divided
  * into uniform chunks of moderate size, which are executed ... in an ascending

@@ -25,7 +25,7 @@ __all__ = [
     "jp_profile_classify", "jp_profile_density", "jp_select_mode", "jp_run_doall", "jp_run_privatized",
     "jp_priv_stream", "jp_priv_finalize", "jp_doall_kernel", "jp_tls_guide", "tls_first_window", "jp_run_tls", "jp_schedule", "jp_stage_bytes", "jp_schedule_host",
     "jp_plan_sharing", "jp_plan_stealing", "jp_merge_apply",
-    "jp_run_doall_spill", "jp_ipc_export", "jp_ipc_import", "jp_ipc_close",
+    "jp_plan_tasks", "jp_export_keys", "jp_run_doall_spill", "jp_ipc_export", "jp_ipc_import", "jp_ipc_close",
     "jp_sparse_scratch_bytes", "jp_sparse_pack", "jp_sparse_reduce_max", "jp_sparse_gather", "jp_sparse_scatter",
     "jp_last_error", "jp_version", "jp_launch_count",
 ]
@@ -331,6 +331,26 @@ def jp_plan_stealing(tasks, world: int, chunk_iters: int, speed=None, speed_tls:
 
 def jp_merge_apply(arr: torch.Tensor, keys: torch.Tensor, stream=None):
     check(lib().jp_merge_apply(arr.data_ptr(), arr.numel(), keys.data_ptr(), _stream(stream)))
+
+
+# ---- task stealing across ranks (jp.h) -------------------------------------
+def jp_plan_tasks(loop: Loop, chunk_counts, chunk_iters: int, ws, tau_high: float = 0.25, stream=None):
+    """chunk_counts: the whole loop's (raw, war, waw) per chunk (flat list / int64
+    tensor).  Returns ([(start, end, mode)], conf list of 64 ints)."""
+    cc = [int(x) for x in (chunk_counts.tolist() if hasattr(chunk_counts, "tolist") else chunk_counts)]
+    hc = (C.c_int64 * max(len(cc), 1))(*cc)
+    tk = (C.c_int64 * 192)()
+    nt = C.c_int32()
+    cf = (C.c_uint64 * 64)()
+    p, nb = _ws(ws)
+    check(lib().jp_plan_tasks(loop.ref, hc, int(chunk_iters), float(tau_high), p, nb, tk, C.byref(nt), cf,
+                              _stream(stream)))
+    return [(tk[3 * t], tk[3 * t + 1], tk[3 * t + 2]) for t in range(nt.value)], list(cf)
+
+
+def jp_export_keys(loop: Loop, ws, stream=None):
+    p, nb = _ws(ws)
+    check(lib().jp_export_keys(loop.ref, p, nb, _stream(stream)))
 
 
 # ---- task sharing with cross-boundary spill (jp.h, M1 / C8) --------------

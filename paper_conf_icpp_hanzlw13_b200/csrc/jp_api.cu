@@ -956,6 +956,60 @@ struct StreamPool {
 } g_pool;
 }  // namespace
 
+
+// ---- task-stealing helpers (shared by jp_schedule(STEALING) and jp_plan_tasks) ----
+struct Task { int64_t s, e; int mode; };
+
+// chunk modes (Fig. 2(b) on each chunk's counts, reading A19) -> maximal same-mode
+// runs, coarsened to <= kMaxTasks by merging the smallest adjacent pair into the
+// stronger mode
+static std::vector<Task> chunk_tasks(const int64_t *hc, int64_t n, int64_t chunk, double tau) {
+  std::vector<Task> tasks;
+  const int64_t nck = (n + chunk - 1) / chunk;
+  for (int64_t k = 0; k < nck; k++) {
+    const int64_t s = k * chunk, e = std::min(n, s + chunk);
+    int m = select_mode_counts(e - s, hc[3 * k], hc[3 * k + 1], hc[3 * k + 2], tau);
+    if (m == JP_MODE_SEQ_RECOMMENDED) m = JP_MODE_TLS;
+    if (!tasks.empty() && tasks.back().mode == m) tasks.back().e = e;
+    else tasks.push_back({s, e, m});
+  }
+  auto rank = [](int m) { return m == JP_MODE_TLS ? 2 : m == JP_MODE_PRIVATIZED ? 1 : 0; };
+  while ((int)tasks.size() > kMaxTasks) {
+    size_t best = 0;
+    for (size_t q = 1; q + 1 < tasks.size(); q++)
+      if (tasks[q].e - tasks[q].s + tasks[q + 1].e - tasks[q + 1].s <
+          tasks[best].e - tasks[best].s + tasks[best + 1].e - tasks[best + 1].s) best = q;
+    tasks[best].e = tasks[best + 1].e;
+    if (rank(tasks[best + 1].mode) > rank(tasks[best].mode)) tasks[best].mode = tasks[best + 1].mode;
+    tasks.erase(tasks.begin() + best + 1);
+  }
+  return tasks;
+}
+
+// conf[u] bit t: tasks t and u touch a common address, at least one writing it (reading B2); syncs
+static jp_status task_conflicts(const Job &j, const jp_loop *L, void *ws, const Layout &lo,
+                                const std::vector<Task> &tasks, int64_t chunk, std::vector<unsigned long long> &conf,
+                                cudaStream_t st) {
+  const int nt = (int)tasks.size();
+  conf.assign(kMaxTasks, 0);
+  if (nt <= 1) return JP_OK;
+  SchedLayout sl = sched_layout(L);
+  char *sch = static_cast<char *>(ws) + lo.off[R_SCHED];
+  const int64_t nck = (L->n + chunk - 1) / chunk;
+  std::vector<int32_t> ct(nck);
+  for (int t = 0; t < nt; t++)
+    for (int64_t k = tasks[t].s / chunk; k * chunk < tasks[t].e; k++) ct[k] = t;
+  int32_t *dct = reinterpret_cast<int32_t *>(sch + sl.chunk_task);
+  JP_CUDA(cudaMemcpyAsync(dct, ct.data(), 4 * nck, cudaMemcpyHostToDevice, st), "task map H2D");
+  auto P = [&](size_t o) { return o == SIZE_MAX ? nullptr : reinterpret_cast<unsigned long long *>(sch + o); };
+  unsigned long long *dconf = P(sl.conf);
+  JP_CUDA(launch_task_conflicts(j, dct, chunk, nt, P(sl.wmA), P(sl.rmA), P(sl.wmT), P(sl.rmT), dconf, st),
+          "conflicts");
+  JP_CUDA(cudaMemcpyAsync(conf.data(), dconf, 8 * kMaxTasks, cudaMemcpyDeviceToHost, st), "conf D2H");
+  JP_CUDA(cudaStreamSynchronize(st), "conf sync");
+  return JP_OK;
+}
+
 static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sched_cfg &c, void *ws, size_t ws_bytes,
                                    jp_sched_result *res, cudaStream_t st) {
   const int64_t chunk = c.chunk_iters;
@@ -982,44 +1036,13 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
   fill_profile(&res->prof, L->n, h.data());
   res->profiled = 1;
   // 2. chunk modes -> tasks (maximal same-mode runs)
-  struct Task { int64_t s, e; int mode; };
-  std::vector<Task> tasks;
-  for (int64_t k = 0; k < nck; k++) {
-    const int64_t s = k * chunk, e = std::min(L->n, s + chunk);
-    int m = select_mode_counts(e - s, hc[3 * k], hc[3 * k + 1], hc[3 * k + 2], c.tau_high);
-    if (m == JP_MODE_SEQ_RECOMMENDED) m = JP_MODE_TLS;
-    if (!tasks.empty() && tasks.back().mode == m) tasks.back().e = e;
-    else tasks.push_back({s, e, m});
-  }
-  // coarsen to <= 64 tasks: merge the smallest adjacent pair into the stronger mode
-  auto rank = [](int m) { return m == JP_MODE_TLS ? 2 : m == JP_MODE_PRIVATIZED ? 1 : 0; };
-  while ((int)tasks.size() > kMaxTasks) {
-    size_t best = 0;
-    for (size_t q = 1; q + 1 < tasks.size(); q++)
-      if (tasks[q].e - tasks[q].s + tasks[q + 1].e - tasks[q + 1].s <
-          tasks[best].e - tasks[best].s + tasks[best + 1].e - tasks[best + 1].s) best = q;
-    tasks[best].e = tasks[best + 1].e;
-    if (rank(tasks[best + 1].mode) > rank(tasks[best].mode)) tasks[best].mode = tasks[best + 1].mode;
-    tasks.erase(tasks.begin() + best + 1);
-  }
+  std::vector<Task> tasks = chunk_tasks(hc.data(), L->n, chunk, c.tau_high);
   const int nt = (int)tasks.size();
   res->n_tasks = nt;
   res->mode = nt ? tasks[0].mode : JP_MODE_DOALL;
   // 3. inter-task conflicts (PDG) and topological batches
   std::vector<unsigned long long> conf(kMaxTasks, 0);
-  if (nt > 1) {
-    std::vector<int32_t> ct(nck);
-    for (int t = 0; t < nt; t++)
-      for (int64_t k = tasks[t].s / chunk; k * chunk < tasks[t].e; k++) ct[k] = t;
-    int32_t *dct = reinterpret_cast<int32_t *>(sch + sl.chunk_task);
-    JP_CUDA(cudaMemcpyAsync(dct, ct.data(), 4 * nck, cudaMemcpyHostToDevice, st), "task map H2D");
-    auto P = [&](size_t o) { return o == SIZE_MAX ? nullptr : reinterpret_cast<unsigned long long *>(sch + o); };
-    unsigned long long *dconf = P(sl.conf);
-    JP_CUDA(launch_task_conflicts(j, dct, chunk, nt, P(sl.wmA), P(sl.rmA), P(sl.wmT), P(sl.rmT), dconf, st),
-            "conflicts");
-    JP_CUDA(cudaMemcpyAsync(conf.data(), dconf, 8 * kMaxTasks, cudaMemcpyDeviceToHost, st), "conf D2H");
-    JP_CUDA(cudaStreamSynchronize(st), "conf sync");
-  }
+  JP_TRY(task_conflicts(j, L, ws, lo, tasks, chunk, conf, st));
   std::vector<int> level(nt, 0);
   int nlev = nt ? 1 : 0;
   for (int u = 0; u < nt; u++) {
@@ -1137,6 +1160,38 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
   JP_CUDA(cudaStreamSynchronize(st), "schedule sync");
   cudaEventDestroy(ev0);
   for (auto e : evs) cudaEventDestroy(e);
+  return JP_OK;
+}
+
+jp_status jp_plan_tasks(const jp_loop *L, const int64_t *chunk_counts, int64_t chunk_iters, double tau_high,
+                        void *ws, size_t ws_bytes, int64_t *tasks, int32_t *n_tasks, uint64_t *conf,
+                        jp_stream_t st) {
+  JP_TRY(check_loop(L));
+  if (!chunk_counts || !tasks || !n_tasks || !conf) return fail(JP_ERR_ARG, "NULL output or counts");
+  if (chunk_iters < kSchedMinChunk || chunk_iters % 32)
+    return fail(JP_ERR_ARG, "chunk_iters must be >= 1024 and a multiple of 32");
+  JP_TRY(need_device());
+  Layout lo;
+  JP_TRY(check_ws(L, ws, ws_bytes, JP_WS_ALL, lo));
+  std::vector<Task> tk = chunk_tasks(chunk_counts, L->n, chunk_iters, tau_high > 0.0 ? tau_high : 0.25);
+  std::vector<unsigned long long> cf;
+  JP_TRY(task_conflicts(make_job(L), L, ws, lo, tk, chunk_iters, cf, (cudaStream_t)st));
+  *n_tasks = (int32_t)tk.size();
+  for (size_t t = 0; t < tk.size(); t++) {
+    tasks[3 * t] = tk[t].s;
+    tasks[3 * t + 1] = tk[t].e;
+    tasks[3 * t + 2] = tk[t].mode;
+  }
+  for (int t = 0; t < kMaxTasks; t++) conf[t] = cf[t];
+  return JP_OK;
+}
+
+jp_status jp_export_keys(const jp_loop *L, void *ws, size_t ws_bytes, jp_stream_t st) {
+  JP_TRY(check_loop(L));
+  JP_TRY(need_device());
+  Layout lo;
+  JP_TRY(check_ws(L, ws, ws_bytes, JP_WS_PRIV, lo));
+  JP_CUDA(launch_export_keys(make_job(L), ws, lo, (cudaStream_t)st), "export keys");
   return JP_OK;
 }
 

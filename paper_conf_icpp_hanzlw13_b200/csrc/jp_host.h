@@ -62,6 +62,8 @@ cudaError_t launch_priv_stream(const Job &j, void *ws, const Layout &lo, bool cl
                                cudaStream_t st, int max_ctas = 0, bool fuse_apply = false, bool *applied = nullptr);
 cudaError_t launch_priv_finalize(const Job &j, void *ws, const Layout &lo, cudaStream_t st);
 cudaError_t launch_merge_apply(void *arr, int64_t len, const int64_t *keys, cudaStream_t st);
+// keys (regions 5/6) of what loop j already wrote in place (atomicMax, keys not cleared)
+cudaError_t launch_export_keys(const Job &j, void *ws, const Layout &lo, cudaStream_t st);
 // task sharing with cross-boundary spill (jp_doall.cu, C8): views[k] = rank k's affine shard
 constexpr int kSpillRanks = 8;
 cudaError_t launch_doall_spill(const Job *views, int world, int me, int64_t chunk, unsigned long long *ctr,

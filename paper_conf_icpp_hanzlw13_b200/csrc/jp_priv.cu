@@ -326,6 +326,42 @@ cudaError_t launch_priv_finalize(const Job &j, void *ws, const Layout &lo, cudaS
   return launch_check();
 }
 
+// Packed last-writer keys of what a loop (or a range of one) has ALREADY written
+// in place, e.g. a TLS task of the multi-rank stealing scheme: every writer of
+// address a offers (gid+1) << 32 | (current value of a), so the max is the last
+// writer's key carrying the final value (reading A9).  Keys only for the arrays
+// that have a key table (indirect writes); identity outputs stay where they are.
+template <int OP, int DT>
+__global__ void __launch_bounds__(256) k_export_keys(DLoop L, unsigned long long *kA, unsigned long long *kT) {
+  const int64_t stride = (int64_t)gridDim.x * blockDim.x;
+  for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < L.n; i += stride) {
+    if (kA) {
+      const int64_t a = ixl(L, L.w, i);
+      atomicMax(&kA[a], pack_key(L.base + i, __ldcg(L.A + a)));
+    }
+    if constexpr (OP == JP_OP_PRIV_TMP) {
+      if (kT) {
+        const int64_t b = ixl(L, L.s, i);
+        atomicMax(&kT[b], pack_key(L.base + i, __ldcg(L.T + b)));
+      }
+    }
+  }
+}
+
+template <int OP, int DT>
+static void run_export(const DLoop &d, unsigned long long *kA, unsigned long long *kT, cudaStream_t st) {
+  int64_t need = (d.n + 255) / 256, cap = (int64_t)num_sms() * 8;
+  k_export_keys<OP, DT><<<(int)(need < cap ? need : cap), 256, 0, st>>>(d, kA, kT);
+  note_launch();
+}
+
+cudaError_t launch_export_keys(const Job &j, void *ws, const Layout &lo, cudaStream_t st) {
+  if (j.d.n == 0) return cudaSuccess;
+  JP_DISPATCH(j.op, j.dt, run_export, j.d, at<unsigned long long>(ws, lo, R_KEYS_A),
+              at<unsigned long long>(ws, lo, R_KEYS_T), st);
+  return launch_check();
+}
+
 cudaError_t launch_merge_apply(void *arr, int64_t len, const int64_t *keys, cudaStream_t st) {
   apply(static_cast<uint32_t *>(arr), len, reinterpret_cast<const unsigned long long *>(keys), st);
   return launch_check();

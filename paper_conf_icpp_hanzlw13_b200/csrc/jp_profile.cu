@@ -220,10 +220,13 @@ __global__ void __launch_bounds__(256) k_prof_count4(DLoop L, Tabs t, int vec, i
           const int32_t a = q4(va[u], k);
           bool raw = false, war, waw;
           if constexpr (OP == JP_OP_ADD_C) {
-            raw = earlier32(t.wA, q4(vb[u], k), lenA, e);
+            // r == w (an in-place update, most iterations of configs 3 and 5):
+            // the raw and waw lookups are the same table entry -- one load
+            const int32_t b = q4(vb[u], k);
             war = earlier32(t.rA, a, lenA, e);
             waw = earlier32(t.wA, a, lenA, e);
-            if (raw) mark_src(q4(vb[u], k));
+            raw = b == a ? waw : earlier32(t.wA, b, lenA, e);
+            if (raw) mark_src(b);
           } else if constexpr (OP == JP_OP_SAXPY) {
             raw = earlier32(t.wA, a, lenA, e);
             war = earlier32(t.rA, a, lenA, e);
@@ -233,10 +236,12 @@ __global__ void __launch_bounds__(256) k_prof_count4(DLoop L, Tabs t, int vec, i
             war = earlier32(rT, a, lenT, e);
             waw = earlier32(t.wT, a, lenT, e) || earlier32(t.wA, q4(vb[u], k), lenA, e);
           } else {
-            const bool r0 = earlier32(t.wA, q4(vb[u], k), lenA, e), r1 = earlier32(t.wA, q4(vc[u], k), lenA, e);
-            raw = r0 || r1;
             war = earlier32(t.rA, a, lenA, e);
             waw = earlier32(t.wA, a, lenA, e);
+            const int32_t b = q4(vb[u], k), c = q4(vc[u], k);
+            const bool r0 = b == a ? waw : earlier32(t.wA, b, lenA, e);
+            const bool r1 = c == a ? waw : c == b ? r0 : earlier32(t.wA, c, lenA, e);
+            raw = r0 || r1;
             if (r0) mark_src(q4(vb[u], k));
             if (r1) mark_src(q4(vc[u], k));
           }
@@ -327,9 +332,9 @@ __global__ void __launch_bounds__(256) k_prof_classify(DLoop L, Tabs t, uint32_t
           }
         };
         if constexpr (OP == JP_OP_ADD_C) {
-          raw[u] = earlier(t.wA, ib[u], L.lenA, e);
           war[u] = earlier(t.rA, ia[u], L.lenA, e);
           waw[u] = earlier(t.wA, ia[u], L.lenA, e);
+          raw[u] = ib[u] == ia[u] ? waw[u] : earlier(t.wA, ib[u], L.lenA, e);   // r == w: one lookup
           if (raw[u]) src(ib[u]);
         } else if constexpr (OP == JP_OP_SAXPY) {
           raw[u] = earlier(t.wA, ia[u], L.lenA, e);
@@ -340,10 +345,11 @@ __global__ void __launch_bounds__(256) k_prof_classify(DLoop L, Tabs t, uint32_t
           war[u] = earlier(rT, ia[u], L.lenT, e);
           waw[u] = earlier(t.wT, ia[u], L.lenT, e) || earlier(t.wA, ib[u], L.lenA, e);
         } else {
-          const bool r0 = earlier(t.wA, ib[u], L.lenA, e), r1 = earlier(t.wA, ic[u], L.lenA, e);
-          raw[u] = r0 || r1;
           war[u] = earlier(t.rA, ia[u], L.lenA, e);
           waw[u] = earlier(t.wA, ia[u], L.lenA, e);
+          const bool r0 = ib[u] == ia[u] ? waw[u] : earlier(t.wA, ib[u], L.lenA, e);
+          const bool r1 = ic[u] == ia[u] ? waw[u] : ic[u] == ib[u] ? r0 : earlier(t.wA, ic[u], L.lenA, e);
+          raw[u] = r0 || r1;
           if (r0) src(ib[u]);
           if (r1) src(ic[u]);
         }

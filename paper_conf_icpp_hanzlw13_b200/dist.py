@@ -134,7 +134,8 @@ def _reduce_tables(tabs, empty, group, exchange, jp):
     return []
 
 
-def profile_partitioned(loop, ws, group=None, engine=None, exchange: str = "dense") -> dict:
+def profile_partitioned(loop, ws, group=None, engine=None, exchange: str = "dense", chunk_iters: int = 0,
+                        chunk_counts=None) -> dict:
     """Profile of the whole loop from rank-local ranges (iter_base = global id of
     the rank's first iteration): stamp locally, C1 (dense or owner form),
     classify locally, C3.  The result equals the single-GPU profile exactly
@@ -148,7 +149,10 @@ def profile_partitioned(loop, ws, group=None, engine=None, exchange: str = "dens
         if left:
             owner_reduce_touched(left[0], left[1] if len(left) > 1 else None, -1, group, jp)
         _reduce_tables([_region(ws, loop, n, torch.int32, jp) for n in ("minW_T", "minR_T")], -1, group, "dense", jp)
-    p = jp.jp_profile_classify(loop, ws)
+    if chunk_counts is None:
+        p = jp.jp_profile_classify(loop, ws)
+    else:
+        p = jp.jp_profile_classify(loop, ws, chunk_iters=chunk_iters, chunk_counts=chunk_counts)
     if world > 1:
         dev = ws.device
         c = torch.tensor([p["n"], p["raw_iters"], p["war_iters"], p["waw_iters"]], dtype=torch.int64, device=dev)
@@ -219,6 +223,103 @@ def schedule_partitioned(loop, ws, group=None, tau_high: float = 0.25, tls_windo
                 if t is not None:
                     dist.broadcast(t, src=0, group=group)
     return res
+
+
+def _levels(conf, nt):
+    """Topological batch of every task: 1 + the highest batch it depends on."""
+    lv = [0] * nt
+    for u in range(nt):
+        for t in range(u):
+            if (conf[u] >> t) & 1:
+                lv[u] = max(lv[u], lv[t] + 1)
+    return lv
+
+
+def schedule_stealing(full, ws, group=None, chunk_iters: int = 65536, tau_high: float = 0.25, speed=None,
+                      speed_tls: float = 1.0, exchange: str = "dense", engine=None) -> dict:
+    """Task stealing of one loop across the ranks (Alg. 1; SURVEY
+    Sec.8(e) "Mixed").  Every rank holds full replicas (``full``, workspace
+    ``ws`` of the whole loop):
+
+      1. partitioned profile with per-chunk counts: rank k stamps its
+         chunk-aligned range, C1, classifies its chunks, then C3 (SUM) of the
+         whole chunk-count array and of the totals;
+      2. jp_plan_tasks on every rank (identical): tasks = maximal same-mode chunk
+         runs, PDG from the per-address task masks (reading B2), batches;
+      3. jp_plan_stealing: chunk owners by Alg. 1 (TLS tasks pinned to rank 0,
+         tails stolen by idle ranks, reading A18);
+      4. batch by batch: each rank runs its chunks -- DOALL / PRIVATIZED chunks
+         through the privatized stream (packed last-writer keys; their exposed
+         reads see the replica, which holds every earlier batch), rank 0 the
+         batch's TLS tasks in place (then jp_export_keys) -- then C4 over the
+         keys (dense or owner form) and every rank applies them: every replica
+         holds the sequential result after the last batch.  Outputs written
+         through identity indices (no key table, e.g. config 4's Y) stay with
+         the rank that executed the chunk, as under task sharing (``chunks``
+         of the result gives the owners).
+    """
+    jp = _engine(engine)
+    world, rank = world_rank(group)
+    n = full.n
+    nck = -(-n // chunk_iters)
+    c0, c1 = rank * nck // world, (rank + 1) * nck // world
+    b, e = min(c0 * chunk_iters, n), min(c1 * chunk_iters, n)
+    loop = full.range(b, e)
+    dev = ws.device
+    cc_loc = torch.zeros(max(3 * (c1 - c0), 3), dtype=torch.int64, device=dev)
+    prof = profile_partitioned(loop, ws, group, jp, exchange, chunk_iters, cc_loc)
+    cc = torch.zeros(3 * nck, dtype=torch.int64, device=dev)
+    cc[3 * c0:3 * c1] = cc_loc[:3 * (c1 - c0)]
+    if world > 1:
+        dist.all_reduce(cc, group=group)
+    tasks, conf = jp.jp_plan_tasks(full, cc.cpu(), chunk_iters, ws, tau_high)
+    lv = _levels(conf, len(tasks))
+    chunks, stolen = jp.jp_plan_stealing(tasks, world, chunk_iters, speed, speed_tls)
+    task_of = {}
+    for t, (s, e2, _) in enumerate(tasks):
+        task_of[(s, e2)] = t
+    ccl = cc.cpu().tolist()
+    tls_stats = {"committed": 0, "executed": 0, "windows": 0, "violations": 0}
+    mine = {"chunks": 0, "iters": 0}
+    for level in range(max(lv) + 1 if lv else 0):
+        for name in ("keys_A", "keys_T"):
+            t = _region(ws, full, name, torch.int64, jp)
+            if t is not None:
+                t.zero_()
+        for t, (s, e2, mode) in enumerate(tasks):
+            if lv[t] != level:
+                continue
+            if mode in (_abi.JP_MODE_TLS, _abi.JP_MODE_SEQ_RECOMMENDED):
+                if rank == 0:   # pinned (Alg. 1: TLS tasks are never stolen)
+                    sub = full.range(s, e2)
+                    k0, k1 = s // chunk_iters, -(-e2 // chunk_iters)
+                    raw = sum(ccl[3 * k] for k in range(k0, k1))
+                    waw = sum(ccl[3 * k + 2] for k in range(k0, k1))
+                    tp = {"n": e2 - s, "raw_iters": raw, "war_iters": 0, "waw_iters": waw, "first_raw_iter": -1,
+                          "d_raw": raw / max(e2 - s, 1), "d_war": 0.0, "d_waw": waw / max(e2 - s, 1)}
+                    st = jp.jp_run_tls(sub, prof=tp, ws=ws, recovery=int(waw == 0))
+                    for k in tls_stats:
+                        tls_stats[k] += st[k]
+                    jp.jp_export_keys(sub, ws)
+                    mine["chunks"] += k1 - k0
+                    mine["iters"] += e2 - s
+                continue
+            for (cs, ce, cm, owner) in chunks:
+                if owner == rank and s <= cs and ce <= e2:
+                    jp.jp_priv_stream(full.range(cs, ce), _NO_RAW, ws, clear_keys=False)
+                    mine["chunks"] += 1
+                    mine["iters"] += ce - cs
+        if world > 1:
+            for name in ("keys_A", "keys_T"):
+                for t in _reduce_tables([_region(ws, full, name, torch.int64, jp)], 0, group, exchange, jp):
+                    owner_reduce_replicate(t, 0, group, jp)
+        jp.jp_priv_finalize(full, ws)
+    return {"scheme": "stealing", "prof": prof, "n_tasks": len(tasks), "n_batches": max(lv) + 1 if lv else 0,
+            "tasks": tasks, "chunks": chunks, "stolen": stolen, "tls": tls_stats, "rank_work": mine}
+
+
+_NO_RAW = {"n": 0, "raw_iters": 0, "war_iters": 0, "waw_iters": 0, "first_raw_iter": -1, "d_raw": 0.0, "d_war": 0.0,
+           "d_waw": 0.0}
 
 
 class SpillGroup:

@@ -71,8 +71,11 @@ def jp_profile_stamp(loop, ws):
                 tab[a] = max(tab[a], e)
 
 
-def jp_profile_classify(loop, ws):
+def jp_profile_classify(loop, ws, chunk_iters=0, chunk_counts=None, **kw):
     ind = _indirect(loop)
+    if chunk_counts is not None:
+        chunk_counts.zero_()
+    cc = None if chunk_counts is None else chunk_counts.numpy()
     tabs = {k: _view(ws, loop, k, torch.int32) for k in ("minW_A", "minR_A", "minW_T", "minR_T")}
     raw = war = waw = 0
     first = -1
@@ -91,6 +94,11 @@ def jp_profile_classify(loop, ws):
         raw += fr
         war += fa
         waw += fw
+        if cc is not None:
+            c = i // chunk_iters
+            cc[3 * c] += fr
+            cc[3 * c + 1] += fa
+            cc[3 * c + 2] += fw
         if fr and first < 0:
             first = loop.iter_base + i
     n = loop.n
@@ -174,7 +182,14 @@ def jp_schedule(loop, ws=None, **kw):
     return {"mode": 0, "mode_name": "DOALL", "profiled": 0}
 
 
-def jp_run_tls(loop, window=0, w_max=65536, path=0, prof=None, ws=None, stats=True):
+def jp_run_tls(loop, window=0, w_max=65536, path=0, prof=None, ws=None, stats=True, **kw):
+    if loop.ident_off or loop.iter_base:   # a range of a loop: its committed result is the in-order one
+        t = loop.tensors
+        ix = lambda a, i: loop.ident_off + i if a is None else int(a[i])  # noqa: E731
+        for i in range(loop.n):
+            for arr, v in _values(loop, i, _np(t["A"]), _np(t["X"])).items():
+                _np(t[arr])[ix(t["w"], i) if arr == "A" else ix(t["s"], i)] = v
+        return {"committed": loop.n, "executed": loop.n, "windows": 1, "violations": 0}
     st, A, T, stats_ = O.sim_tls(_oracle_loop(loop), window, w_max, -1 if prof is None else prof["raw_iters"])
     assert st == 0
     _np(loop.tensors["A"])[:] = A
@@ -223,3 +238,48 @@ def jp_sparse_scatter(t0, t1, rows):
     for q, t in enumerate([t0, t1]):
         if t is not None:
             t.numpy()[a[ok]] = rows.numpy()[ok, 1 + q]
+
+
+# ---- task stealing across ranks (jp.h jp_plan_tasks / jp_export_keys), plain definitions ----
+def jp_plan_tasks(loop, chunk_counts, chunk_iters, ws, tau_high=0.25):
+    import oracle.sched as OS
+    cc = [int(x) for x in (chunk_counts.tolist() if hasattr(chunk_counts, "tolist") else chunk_counts)]
+    n = loop.n
+    tasks = []
+    for k in range(-(-n // chunk_iters)):
+        s, e = k * chunk_iters, min(n, (k + 1) * chunk_iters)
+        m = OS.select_mode(False, e - s, cc[3 * k], cc[3 * k + 1], cc[3 * k + 2], tau_high)
+        m = OS.TLS if m == OS.SEQ_RECOMMENDED else m
+        if tasks and tasks[-1][2] == m:
+            tasks[-1][1] = e
+        else:
+            tasks.append([s, e, m])
+    assert len(tasks) <= 64
+    sets = []
+    for s, e, _ in tasks:
+        wr, rd = set(), set()
+        for i in range(s, e):
+            for arr, a, kind in _accesses(loop, i):
+                (wr if kind == "w" else rd).add((arr, a))
+        sets.append((wr, rd))
+    conf = [0] * 64
+    for u in range(len(tasks)):
+        for t in range(u):
+            (wt, rt), (wu, ru) = sets[t], sets[u]
+            if wt & (wu | ru) or rt & wu:
+                conf[u] |= 1 << t
+    return [tuple(x) for x in tasks], conf
+
+
+def jp_export_keys(loop, ws):
+    ind = _indirect(loop)
+    t = loop.tensors
+    ix = lambda a, i: loop.ident_off + i if a is None else int(a[i])  # noqa: E731
+    for arr in ("A", "T"):
+        k = _view(ws, loop, "keys_" + arr, torch.int64)
+        if k is None or not ind[arr] or (arr == "T" and loop.op != O.OP_PRIV_TMP):
+            continue
+        for i in range(loop.n):
+            a = ix(t["w"], i) if arr == "A" else ix(t["s"], i)
+            key = ((loop.iter_base + i + 1) << 32) | int(_np(t[arr]).view(np.uint32)[a])
+            k[a] = max(int(k[a]), key)

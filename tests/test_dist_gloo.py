@@ -107,3 +107,51 @@ def test_sharing_ranges_cover_and_match_plan():
     chunks, stolen = jd.stealing_plan([(0, 1 << 20, 2), (1 << 20, 1 << 22, 0)], 4, 1 << 16, engine=fe)
     assert all(c[3] == 0 for c in chunks if c[2] == 2)
     assert np.sum([c[1] - c[0] for c in chunks]) == 1 << 22
+
+
+def _steal_worker(rank, world, port, case, exchange, q):
+    sys.path[:0] = [ROOT, os.path.join(ROOT, "tests")]
+    os.environ.update(MASTER_ADDR="127.0.0.1", MASTER_PORT=str(port))
+    dist.init_process_group("gloo", rank=rank, world_size=world)
+    try:
+        import fake_engine as fe
+        import oracle as O
+        import paper_conf_icpp_hanzlw13_b200 as jp
+        from paper_conf_icpp_hanzlw13_b200 import dist as jd
+        import synth
+        from helpers import to_oracle
+        wl = {"c5": lambda: synth.config5(n=1 << 12, delta=64),
+              "c1_5": lambda: synth.config1(0.05, n=4096)}[case]()
+        ref = to_oracle(wl)
+        _, A_exp, _ = O.run_seq(ref)
+        full = jp.Loop.from_workload(wl)
+        ws = torch.zeros(jp.jp_workspace_bytes(full), dtype=torch.uint8)
+        jd.OWNER_MIN_LEN = 0
+        res = jd.schedule_stealing(full, ws, chunk_iters=1024, exchange=exchange, engine=fe)
+        ok = wl.A.numpy().tobytes() == A_exp.tobytes()
+        q.put((rank, bool(ok), res["n_tasks"], res["n_batches"], res["rank_work"]["iters"]))
+    except Exception:  # pragma: no cover
+        import traceback
+        q.put((rank, False, traceback.format_exc(), 0, 0))
+    finally:
+        dist.destroy_process_group()
+
+
+@pytest.mark.parametrize("exchange", ["dense", "owner"])
+@pytest.mark.parametrize("world", [2, 3])
+@pytest.mark.parametrize("case", ["c5", "c1_5"])
+def test_stealing_scheme_matches_oracle(case, world, exchange):
+    """Multi-rank task stealing (dist.schedule_stealing): partitioned profile with
+    chunk counts, tasks + PDG, Alg. 1 plan, batches with C4 merges; every
+    replica ends with the oracle's sequential result."""
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    port = _free_port()
+    ps = [ctx.Process(target=_steal_worker, args=(r, world, port, case, exchange, q)) for r in range(world)]
+    for p in ps:
+        p.start()
+    out = sorted(q.get(timeout=300) for _ in range(world))
+    for p in ps:
+        p.join(timeout=60)
+    assert [o[1] for o in out] == [True] * world, out
+    assert sum(o[4] for o in out) == 4096

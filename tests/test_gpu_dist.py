@@ -79,3 +79,59 @@ def test_two_ranks_one_gpu(case, mode, exchange):
         p.join(timeout=120)
     assert [o[1] for o in out] == [True, True], out
     assert all(o[2] == mode for o in out), out
+
+
+def _steal_worker(rank, world, port, case, exchange, q):
+    sys.path[:0] = [ROOT, os.path.join(ROOT, "tests")]
+    os.environ.update(MASTER_ADDR="127.0.0.1", MASTER_PORT=str(port))
+    dist.init_process_group("gloo", rank=rank, world_size=world)
+    try:
+        import oracle as O
+        import paper_conf_icpp_hanzlw13_b200 as jp
+        from paper_conf_icpp_hanzlw13_b200 import dist as jd
+        import synth
+        from helpers import to_oracle
+        wl = {"c5": lambda: synth.config5(n=1 << 18), "c5big": lambda: synth.config5(n=1 << 20, density=0.01),
+              "c4": lambda: synth.config4(n=(1 << 18) + 64, slots=1024)}[case]()
+        ref = to_oracle(wl)
+        _, A_exp, T_exp = O.run_seq(ref)
+        g = wl.to("cuda:0")
+        full = jp.Loop.from_workload(g)
+        ws = jp.workspace(full)
+        jd.OWNER_MIN_LEN = 1 << 12
+        res = jd.schedule_stealing(full, ws, chunk_iters=1 << 14, exchange=exchange)
+        torch.cuda.synchronize()
+        if wl.op == O.OP_PRIV_TMP:   # Y identity-written: each rank holds the chunks it ran
+            A = g.A.cpu().numpy()
+            ok = all(A[cs:ce].tobytes() == A_exp[cs:ce].tobytes() for cs, ce, _, ow in res["chunks"] if ow == rank)
+        else:
+            ok = g.A.cpu().numpy().tobytes() == A_exp.tobytes()
+        if wl.T is not None:
+            ok &= g.T.cpu().numpy().tobytes() == T_exp.tobytes()
+        p = O.profile(ref)
+        ok &= (res["prof"]["raw_iters"], res["prof"]["war_iters"], res["prof"]["waw_iters"]) == \
+            (p["raw_iters"], p["war_iters"], p["waw_iters"])
+        q.put((rank, bool(ok), res["n_tasks"], res["n_batches"], res["rank_work"]))
+    except Exception as ex:  # pragma: no cover
+        import traceback
+        q.put((rank, False, traceback.format_exc(), 0, None))
+    finally:
+        dist.destroy_process_group()
+
+
+@pytest.mark.parametrize("exchange", ["dense", "owner"])
+@pytest.mark.parametrize("case", ["c5", "c5big", "c4"])
+def test_stealing_two_ranks_one_gpu(case, exchange):
+    """Config 5 (DOALL head, TLS middle, privatized tail) under the multi-rank
+    task-stealing scheme: every replica ends with the sequential result."""
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    port = _port()
+    ps = [ctx.Process(target=_steal_worker, args=(r, 2, port, case, exchange, q)) for r in range(2)]
+    for p in ps:
+        p.start()
+    out = sorted(q.get(timeout=600) for _ in range(2))
+    for p in ps:
+        p.join(timeout=120)
+    assert [o[1] for o in out] == [True, True], out
+    assert sum(o[4]["iters"] for o in out) == {"c5": 1 << 18, "c5big": 1 << 20, "c4": (1 << 18) + 64}[case]
