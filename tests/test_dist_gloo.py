@@ -28,10 +28,7 @@ def _free_port():
     return p
 
 
-def _worker(rank, world, port, case, q, exchange="dense"):
-    sys.path[:0] = [ROOT, os.path.join(ROOT, "tests")]
-    os.environ.update(MASTER_ADDR="127.0.0.1", MASTER_PORT=str(port))
-    dist.init_process_group("gloo", rank=rank, world_size=world)
+def _sharing_case(rank, world, case, q, exchange="dense"):
     try:
         import fake_engine as fe
         import oracle as O
@@ -70,30 +67,76 @@ def _worker(rank, world, port, case, q, exchange="dense"):
         q.put((rank, bool(prof_ok and ok_A), res["mode_name"]))
     except Exception as ex:  # pragma: no cover - reported to the parent
         q.put((rank, False, repr(ex)))
+
+
+def _group_worker(rank, world, port, jobs, q):
+    """One process group per world size; every job (a test case) runs in it in turn."""
+    sys.path[:0] = [ROOT, os.path.join(ROOT, "tests")]
+    os.environ.update(MASTER_ADDR="127.0.0.1", MASTER_PORT=str(port))
+    dist.init_process_group("gloo", rank=rank, world_size=world)
+    try:
+        for k, (kind, case, exchange) in enumerate(jobs):
+            sub = _Tagged(q, k)
+            if kind == "share":
+                _sharing_case(rank, world, case, sub, exchange)
+            else:
+                _steal_case(rank, world, case, exchange, sub)
+            dist.barrier()
     finally:
         dist.destroy_process_group()
 
 
-def run_world(world, case, exchange="dense"):
-    ctx = mp.get_context("spawn")
-    q = ctx.Queue()
-    port = _free_port()
-    ps = [ctx.Process(target=_worker, args=(r, world, port, case, q, exchange)) for r in range(world)]
-    for p in ps:
-        p.start()
-    out = [q.get(timeout=300) for _ in range(world)]
-    for p in ps:
-        p.join(timeout=60)
-    return sorted(out)
+class _Tagged:
+    def __init__(self, q, k):
+        self.q, self.k = q, k
+
+    def put(self, item):
+        self.q.put((self.k, item))
 
 
-@pytest.mark.parametrize("exchange", ["dense", "owner"])
-@pytest.mark.parametrize("world", [2, 3])
-@pytest.mark.parametrize("case,mode", [("c1_0", "DOALL"), ("c1_5", "TLS"), ("c4", "PRIVATIZED"),
-                                       ("c3", "TLS"), ("c2", None), ("c5tail", "PRIVATIZED"),
-                                       ("c5head", "DOALL")])
+_RESULTS = {}
+
+
+def _jobs(world):
+    share = [("share", c, "dense") for c, _ in _CASES]
+    if world == 3:
+        share += [("share", c, "owner") for c in ("c1_5", "c4", "c5tail", "c5head")]
+    else:
+        share += [("share", "c5tail", "owner")]
+    steal = [("steal", "c5", "dense"), ("steal", "c5", "owner")] + ([("steal", "c1_5", "dense")] if world == 2 else [])
+    return share + steal
+
+
+def run_world(world, kind, case, exchange="dense"):
+    """Results of one case; the whole world-size group runs once and is cached."""
+    if world not in _RESULTS:
+        jobs = _jobs(world)
+        ctx = mp.get_context("spawn")
+        q = ctx.Queue()
+        port = _free_port()
+        ps = [ctx.Process(target=_group_worker, args=(r, world, port, jobs, q)) for r in range(world)]
+        for p in ps:
+            p.start()
+        got = {}
+        for _ in range(world * len(jobs)):
+            k, item = q.get(timeout=600)
+            got.setdefault(jobs[k], []).append(item)
+        for p in ps:
+            p.join(timeout=60)
+        _RESULTS[world] = {j: sorted(v, key=lambda x: x[0]) for j, v in got.items()}
+    return _RESULTS[world][(kind, case, exchange)]
+
+
+_CASES = [("c1_0", "DOALL"), ("c1_5", "TLS"), ("c4", "PRIVATIZED"), ("c3", "TLS"), ("c2", None),
+          ("c5tail", "PRIVATIZED"), ("c5head", "DOALL")]
+
+
+@pytest.mark.parametrize("world,case,mode,exchange",
+                         [(w, c, m, "dense") for w in (2, 3) for c, m in _CASES] +
+                         [(3, c, m, "owner") for c, m in _CASES if c in ("c1_5", "c4", "c5tail", "c5head")] +
+                         [(2, "c5tail", "PRIVATIZED", "owner")])
 def test_partitioned_schedule_matches_oracle(world, case, mode, exchange):
-    out = run_world(world, case, exchange)
+    out = run_world(world, "share", case, exchange)
     assert [o[1] for o in out] == [True] * world, out
     if mode:
         assert all(o[2] == mode for o in out), out
@@ -109,10 +152,7 @@ def test_sharing_ranges_cover_and_match_plan():
     assert np.sum([c[1] - c[0] for c in chunks]) == 1 << 22
 
 
-def _steal_worker(rank, world, port, case, exchange, q):
-    sys.path[:0] = [ROOT, os.path.join(ROOT, "tests")]
-    os.environ.update(MASTER_ADDR="127.0.0.1", MASTER_PORT=str(port))
-    dist.init_process_group("gloo", rank=rank, world_size=world)
+def _steal_case(rank, world, case, exchange, q):
     try:
         import fake_engine as fe
         import oracle as O
@@ -133,25 +173,14 @@ def _steal_worker(rank, world, port, case, exchange, q):
     except Exception:  # pragma: no cover
         import traceback
         q.put((rank, False, traceback.format_exc(), 0, 0))
-    finally:
-        dist.destroy_process_group()
 
 
-@pytest.mark.parametrize("exchange", ["dense", "owner"])
-@pytest.mark.parametrize("world", [2, 3])
-@pytest.mark.parametrize("case", ["c5", "c1_5"])
+@pytest.mark.parametrize("case,world,exchange", [("c5", 2, "dense"), ("c5", 3, "dense"), ("c5", 2, "owner"),
+                                                  ("c5", 3, "owner"), ("c1_5", 2, "dense")])
 def test_stealing_scheme_matches_oracle(case, world, exchange):
     """Multi-rank task stealing (dist.schedule_stealing): partitioned profile with
     chunk counts, tasks + PDG, Alg. 1 plan, batches with C4 merges; every
     replica ends with the oracle's sequential result."""
-    ctx = mp.get_context("spawn")
-    q = ctx.Queue()
-    port = _free_port()
-    ps = [ctx.Process(target=_steal_worker, args=(r, world, port, case, exchange, q)) for r in range(world)]
-    for p in ps:
-        p.start()
-    out = sorted(q.get(timeout=300) for _ in range(world))
-    for p in ps:
-        p.join(timeout=60)
+    out = run_world(world, "steal", case, exchange)
     assert [o[1] for o in out] == [True] * world, out
     assert sum(o[4] for o in out) == 4096
