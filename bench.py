@@ -470,6 +470,38 @@ def partitioned_spill(jp, dev, st, world, rank, steps):
     return out
 
 
+def partitioned_config5(jp, dev, st, world, rank, steps):
+    """Config 5 (mixed, N = 2^24) under the multi-rank task-stealing scheme
+    (dist.schedule_stealing: partitioned profile with chunk counts -> tasks +
+    PDG -> Alg. 1 plan -> batches with C4 merges; TLS pinned to rank 0).  One
+    step = the whole call from pristine replicas; wall clock between barriers,
+    max over ranks."""
+    import synth
+    from paper_conf_icpp_hanzlw13_b200 import dist as jd
+    wl = synth.config5(device=dev)
+    A0 = wl.A.clone()
+    full = jp.Loop.from_workload(wl)
+    ws = jp.workspace(full)
+    ts, res = [], None
+    for k in range(steps + 2):
+        wl.A.copy_(A0)
+        torch.cuda.synchronize()
+        barrier(world)
+        t0 = time.perf_counter()
+        res = jd.schedule_stealing(full, ws, chunk_iters=65536)
+        torch.cuda.synchronize()
+        barrier(world)
+        if k >= 2:
+            ts.append(time.perf_counter() - t0)
+    ms = max_over_ranks(statistics.median(ts) * 1e3, world, dev)
+    out = {"workload": "config5 mixed ADD_C int32 N=2^24, multi-rank task stealing (chunk 2^16)", "ms": ms,
+           "iters_per_s": wl.n / (ms * 1e-3), "n_tasks": res["n_tasks"], "n_batches": res["n_batches"],
+           "rank0_iters": res["rank_work"]["iters"], "tls": res["tls"],
+           "timing": "wall clock between barriers, max over ranks"}
+    del wl, A0, full, ws
+    return out
+
+
 def exchange_cost(jp, dev, st):
     """NEXT-2 on one GPU: rank 0 of 8 of config 3 (d = 1%) and config 5's
     privatized tail: what the owner form sends vs the dense all_reduce, and the
@@ -606,8 +638,10 @@ def run_jp(args):
         torch.cuda.empty_cache()
         spill = partitioned_spill(jp, dev, st, world, rank, 5)
         torch.cuda.empty_cache()
+        steal = partitioned_config5(jp, dev, st, world, rank, 3)
+        torch.cuda.empty_cache()
         if rank == 0:
-            out["partitioned"] = {"config4": part, "config2_spill": spill}
+            out["partitioned"] = {"config4": part, "config2_spill": spill, "config5_stealing": steal}
         if world == 1:
             out["modes"] = modes_sweep(jp, dev, st)
             out["modes"]["exchange_owner"] = exchange_cost(jp, dev, st)

@@ -304,11 +304,17 @@ def schedule_stealing(full, ws, group=None, chunk_iters: int = 65536, tau_high: 
                     mine["chunks"] += k1 - k0
                     mine["iters"] += e2 - s
                 continue
-            for (cs, ce, cm, owner) in chunks:
-                if owner == rank and s <= cs and ce <= e2:
-                    jp.jp_priv_stream(full.range(cs, ce), _NO_RAW, ws, clear_keys=False)
-                    mine["chunks"] += 1
-                    mine["iters"] += ce - cs
+            # this rank's chunks of the task, adjacent ones run as one range (one launch)
+            runs = []
+            for (cs, ce, cm, owner) in sorted(c for c in chunks if c[3] == rank and s <= c[0] and c[1] <= e2):
+                if runs and runs[-1][1] == cs:
+                    runs[-1][1] = ce
+                else:
+                    runs.append([cs, ce])
+                mine["chunks"] += 1
+                mine["iters"] += ce - cs
+            for cs, ce in runs:
+                jp.jp_priv_stream(full.range(cs, ce), _NO_RAW, ws, clear_keys=False)
         if world > 1:
             for name in ("keys_A", "keys_T"):
                 for t in _reduce_tables([_region(ws, full, name, torch.int64, jp)], 0, group, exchange, jp):
