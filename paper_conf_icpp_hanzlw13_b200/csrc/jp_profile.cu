@@ -23,6 +23,12 @@
 namespace jp {
 
 // table bytes stamped per pass (env JP_STAMP_PASS_MB overrides, for measurement)
+// env knob read per call (tests and measurements flip it), default dflt
+static int getenv_int(const char *name, int dflt) {
+  const char *e = getenv(name);
+  return e && e[0] ? atoi(e) : dflt;
+}
+
 static size_t stamp_pass_bytes() {
   const char *e = getenv("JP_STAMP_PASS_MB");
   const long mb = e ? atol(e) : 48;
@@ -31,6 +37,10 @@ static size_t stamp_pass_bytes() {
 
 struct Tabs {
   int32_t *wA, *rA, *wT, *rT;
+  // optional interleaved copy {minW[a], minR[a]} of the A tables (classify only):
+  // the war and waw lookups of a written address then cost one 8-byte access
+  // (one DRAM burst) instead of two in separate 64 MiB tables
+  const int2 *pA;
   int sA, sT;   // pre-aggregate in shared memory
   // stamp pass over an address window [lo, lo + span) only (tables larger than
   // L2 are stamped in several passes, each with an L2-resident working set);
@@ -173,7 +183,11 @@ __global__ void __launch_bounds__(256) k_prof_stamp4(DLoop L, Tabs t, int vec, i
 // address twice (then an address read by a later iteration has exactly one
 // writer, the first), which is the only case a guided TLS run accepts; the
 // caller zeroes them first.
-template <int OP, bool GUIDE>
+__device__ __forceinline__ int2 pair32(const int2 *p, int32_t a, int32_t len) {
+  return (uint32_t)a < (uint32_t)len ? __ldg(p + a) : make_int2(-1, -1);
+}
+
+template <int OP, bool GUIDE, bool PAIRS = false>
 __global__ void __launch_bounds__(256) k_prof_count4(DLoop L, Tabs t, int vec, int64_t *hdr, uint32_t *graw,
                                                      uint32_t *gsrc) {
   __shared__ unsigned long long s_cnt[3];
@@ -223,21 +237,39 @@ __global__ void __launch_bounds__(256) k_prof_count4(DLoop L, Tabs t, int vec, i
             // r == w (an in-place update, most iterations of configs 3 and 5):
             // the raw and waw lookups are the same table entry -- one load
             const int32_t b = q4(vb[u], k);
-            war = earlier32(t.rA, a, lenA, e);
-            waw = earlier32(t.wA, a, lenA, e);
+            if constexpr (PAIRS) {
+              const int2 pa = pair32(t.pA, a, lenA);
+              war = pa.y > e;
+              waw = pa.x > e;
+            } else {
+              war = earlier32(t.rA, a, lenA, e);
+              waw = earlier32(t.wA, a, lenA, e);
+            }
             raw = b == a ? waw : earlier32(t.wA, b, lenA, e);
             if (raw) mark_src(b);
           } else if constexpr (OP == JP_OP_SAXPY) {
-            raw = earlier32(t.wA, a, lenA, e);
-            war = earlier32(t.rA, a, lenA, e);
+            if constexpr (PAIRS) {
+              const int2 pa = pair32(t.pA, a, lenA);
+              raw = pa.x > e;
+              war = pa.y > e;
+            } else {
+              raw = earlier32(t.wA, a, lenA, e);
+              war = earlier32(t.rA, a, lenA, e);
+            }
             waw = raw;
             if (raw) mark_src(a);
           } else if constexpr (OP == JP_OP_PRIV_TMP) {
             war = earlier32(rT, a, lenT, e);
             waw = earlier32(t.wT, a, lenT, e) || earlier32(t.wA, q4(vb[u], k), lenA, e);
           } else {
-            war = earlier32(t.rA, a, lenA, e);
-            waw = earlier32(t.wA, a, lenA, e);
+            if constexpr (PAIRS) {
+              const int2 pa = pair32(t.pA, a, lenA);
+              war = pa.y > e;
+              waw = pa.x > e;
+            } else {
+              war = earlier32(t.rA, a, lenA, e);
+              waw = earlier32(t.wA, a, lenA, e);
+            }
             const int32_t b = q4(vb[u], k), c = q4(vc[u], k);
             const bool r0 = b == a ? waw : earlier32(t.wA, b, lenA, e);
             const bool r1 = c == a ? waw : c == b ? r0 : earlier32(t.wA, c, lenA, e);
@@ -491,6 +523,7 @@ static Tabs tabs_of(const DLoop &d, void *ws, const Layout &lo) {
   t.rT = at<int32_t>(ws, lo, R_MINR_T);
   t.sA = t.wA && d.lenA <= kSmemSlots;
   t.sT = t.wT && d.lenT <= kSmemSlots;
+  t.pA = nullptr;
   return t;
 }
 
@@ -553,16 +586,35 @@ cudaError_t launch_prof_classify(const Job &j, void *ws, const Layout &lo, uint3
   return launch_check();
 }
 
+// pairs[a] = {minW[a], minR[a]}: 16-byte loads of both tables, 16-byte stores
+__global__ void __launch_bounds__(256) k_interleave(const int32_t *w, const int32_t *r, int2 *pairs, int64_t len) {
+  const int64_t stride = (int64_t)gridDim.x * blockDim.x, nq = len >> 2;
+  const int4 *w4 = reinterpret_cast<const int4 *>(w), *r4 = reinterpret_cast<const int4 *>(r);
+  int4 *p4 = reinterpret_cast<int4 *>(pairs);
+  for (int64_t q = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; q < nq; q += stride) {
+    const int4 a = __ldcs(w4 + q), b = __ldcs(r4 + q);
+    p4[2 * q] = make_int4(a.x, b.x, a.y, b.y);
+    p4[2 * q + 1] = make_int4(a.z, b.z, a.w, b.w);
+  }
+  for (int64_t a = 4 * nq + (int64_t)blockIdx.x * blockDim.x + threadIdx.x; a < len; a += stride)
+    pairs[a] = make_int2(w[a], r[a]);
+}
+
 template <int OP, int DT>
 static void run_classify_guide(const DLoop &d, Tabs t, uint32_t *graw, uint32_t *gsrc, int64_t *hdr, cudaStream_t st) {
   (void)DT;
   const int64_t nq = (d.n + 3) / 4;
+  const int g = grid_for((nq + kQuadSteps - 1) / kQuadSteps, 256, 8);
   if constexpr (OP == JP_OP_PRIV_TMP) {   // never guided: counts only
-    k_prof_count4<OP, false><<<grid_for((nq + kQuadSteps - 1) / kQuadSteps, 256, 8), 256, 0, st>>>(d, t, idx_vec(d), hdr,
-                                                                                                 nullptr, nullptr);
+    k_prof_count4<OP, false><<<g, 256, 0, st>>>(d, t, idx_vec(d), hdr, nullptr, nullptr);
   } else {
-    k_prof_count4<OP, true><<<grid_for((nq + kQuadSteps - 1) / kQuadSteps, 256, 8), 256, 0, st>>>(d, t, idx_vec(d), hdr,
-                                                                                                graw, gsrc);
+    if (t.pA) {
+      k_interleave<<<grid_for(d.lenA / 4 + 1, 256, 8), 256, 0, st>>>(t.wA, t.rA, const_cast<int2 *>(t.pA), d.lenA);
+      k_prof_count4<OP, true, true><<<g, 256, 0, st>>>(d, t, idx_vec(d), hdr, graw, gsrc);
+      note_launch();
+    } else {
+      k_prof_count4<OP, true><<<g, 256, 0, st>>>(d, t, idx_vec(d), hdr, graw, gsrc);
+    }
   }
   note_launch();
 }
@@ -577,6 +629,13 @@ cudaError_t launch_prof_classify_guide(const Job &j, void *ws, const Layout &lo,
   cudaMemsetAsync(bits + nw, 0, 4 * (size_t)nw, st);   // source words are OR-ed in
   if (j.d.n == 0) return launch_check();
   Tabs t = tabs_of(j.d, ws, lo);
+  // the TLS write-log region (u64 [len_A], reset by every TLS launch) is free
+  // until TLS runs: it holds the interleaved A tables for this pass when the
+  // tables are large (beyond L2, where the second table's lookup is a DRAM burst)
+  unsigned long long *scratch = at<unsigned long long>(ws, lo, R_TLS_S_A);
+  if (scratch && t.wA && t.rA && !t.sA && j.d.lenA >= (1 << 20) && ((uintptr_t)t.wA & 15) == 0 &&
+      ((uintptr_t)t.rA & 15) == 0 && getenv_int("JP_CLASSIFY_PAIRS", 1))
+    t.pA = reinterpret_cast<const int2 *>(scratch);
   JP_DISPATCH(j.op, j.dt, run_classify_guide, j.d, t, bits, bits + nw, hdr, st);
   return launch_check();
 }

@@ -791,3 +791,25 @@ def test_profile_config3_full_size():
     p = jp.jp_profile_density(L, jp.workspace(L))
     assert (p["raw_iters"], p["war_iters"], p["waw_iters"], p["first_raw_iter"]) == \
         (pr["raw_iters"], pr["war_iters"], pr["waw_iters"], pr["first_raw_iter"])
+
+
+@pytest.mark.parametrize("pairs", ["1", "0"])
+@pytest.mark.parametrize("op", [O.OP_ADD_C, O.OP_SAXPY, O.OP_STENCIL2])
+@pytest.mark.parametrize("seed", [3, 4])
+def test_schedule_profile_interleaved_tables(op, seed, pairs, monkeypatch):
+    """jp_schedule's classify pass on tables beyond 2^20 entries reads an
+    interleaved {minW, minR} copy (JP_CLASSIFY_PAIRS=1, the default) or the two
+    tables (0): the profile equals the oracle's either way, and so does the
+    result of the mode it selects."""
+    monkeypatch.setenv("JP_CLASSIFY_PAIRS", pairs)
+    wl = random_loop(seed * 10 + op, op, O.F32 if op != O.OP_ADD_C else O.I32, 60001, len_a=(1 << 20) + 3)
+    ref = to_oracle(wl)
+    p = O.profile(ref)
+    g = gpu(wl)
+    L = jp.Loop.from_workload(g)
+    res = jp.jp_schedule(L, jp.workspace(L), tls_recovery=1)
+    torch.cuda.synchronize()
+    assert (res["prof"]["raw_iters"], res["prof"]["war_iters"], res["prof"]["waw_iters"],
+            res["prof"]["first_raw_iter"]) == (p["raw_iters"], p["war_iters"], p["waw_iters"], p["first_raw_iter"])
+    _, A, T = O.run_seq(ref)
+    check_arrays(g, A, T)
