@@ -384,11 +384,15 @@ def partitioned_config4(jp, dev, st, world, rank, steps):
     prof_ms = timed(lambda: prof.update(jd.profile_partitioned(loop, ws)), steps)
     mode = jp.jp_select_mode(loop, prof, 0.25)
     ms = timed(lambda: jd.privatized_partitioned(loop, ws, prof), steps)
+    ms_p2p = timed(lambda: jd.privatized_partitioned(loop, ws, prof, exchange="p2p"), steps) if world > 1 else None
     hbm, _ = peaks()
     return {"workload": "config4: PRIV_TMP fp32 N=2^26 S=1024, task sharing; step = privatized stream + C4 + finalize",
             "n": wl.n, "n_per_rank": e - b, "mode": jp.MODE_NAMES[mode], "ms": ms, "iters_per_s": wl.n / (ms * 1e-3),
             "per_rank_frac_of_hbm": BYTES_PER_ITER_PRIV * (e - b) / (ms * 1e-3) / 1e9 / hbm,
-            "profile_ms": prof_ms, "collective": "torch.distributed all_reduce MAX (C4, 8 KiB int64)"}
+            "profile_ms": prof_ms, "collective": "torch.distributed all_reduce MAX (C4, 8 KiB int64)",
+            "ms_p2p_merge": ms_p2p,
+            "p2p_merge": "C4 as jp_keys_merge_p2p: one CTA per rank reads every rank's 8 KiB over NVLink (CUDA IPC), "
+                         "two device-side barriers, keys applied in the same kernel; no NCCL call"}
 
 
 def partitioned_spill(jp, dev, st, world, rank, steps):

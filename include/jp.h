@@ -415,6 +415,23 @@ jp_status jp_export_keys(const jp_loop *L, void *ws, size_t ws_bytes, jp_stream_
  * synchronises and barriers).  Stream-ordered.                               */
 jp_status jp_run_doall_spill(const jp_loop *views /* host [world] */, int32_t world, int32_t me, int64_t chunk,
                              unsigned long long *ctr, int64_t *stats, int32_t max_ctas, jp_stream_t st);
+/* C4 over NVLink peer memory, for small key tables (len <= 16384, e.g. config
+ * 4's 1024 private slots; SURVEY §2c C9's role without NCCL).  Every rank calls
+ * it once per merge, after its privatized stream on the same stream:
+ * peer_keys (host [world]): every rank's key table (this rank's included) as
+ * device pointers valid here (jp_ipc_import); keys: this rank's table; bar: a
+ * uint64 counter visible to every rank (in one rank's memory), zero before the
+ * first call and never reset; epoch: 1, 2, ... (the same on every rank).  One
+ * CTA per rank: a device-side barrier (system-scope atomicAdd + acquire
+ * polling of bar) until every rank's keys are in, the max of every slot over
+ * the ranks, a second barrier until every rank has read, then keys = the
+ * merged table and, when arr is not NULL, arr[a] = lo32(keys[a]) where
+ * keys[a] != 0 (jp_merge_apply's rule, reading A9).  A barrier waiting over
+ * ~4 s sets *err (device int32, caller zeroes) to 1 and abandons the merge.
+ * Stream-ordered.                                                          */
+jp_status jp_keys_merge_p2p(const int64_t *const *peer_keys /* host [world] */, int32_t world, int64_t *keys,
+                            int64_t len, unsigned long long *bar, int64_t epoch, void *arr, int32_t *err,
+                            jp_stream_t st);
 /* CUDA IPC plumbing for the spill (peer shards and the counter table):
  * export: a 64-byte handle (host) of the allocation holding ptr, and ptr's
  * byte offset in it; import (in another process): *ptr = mapped base + offset

@@ -25,7 +25,7 @@ __all__ = [
     "jp_profile_classify", "jp_profile_density", "jp_select_mode", "jp_run_doall", "jp_run_privatized",
     "jp_priv_stream", "jp_priv_finalize", "jp_doall_kernel", "jp_tls_guide", "tls_first_window", "jp_run_tls", "jp_schedule", "jp_stage_bytes", "jp_schedule_host",
     "jp_plan_sharing", "jp_plan_stealing", "jp_merge_apply",
-    "jp_plan_tasks", "jp_export_keys", "jp_run_doall_spill", "jp_ipc_export", "jp_ipc_import", "jp_ipc_close",
+    "jp_plan_tasks", "jp_export_keys", "jp_keys_merge_p2p", "jp_run_doall_spill", "jp_ipc_export", "jp_ipc_import", "jp_ipc_close",
     "jp_sparse_scratch_bytes", "jp_sparse_pack", "jp_sparse_reduce_max", "jp_sparse_gather", "jp_sparse_scatter",
     "jp_last_error", "jp_version", "jp_launch_count",
 ]
@@ -362,6 +362,14 @@ def jp_run_doall_spill(views, me: int, chunk: int, ctr: torch.Tensor, stats=None
     arr = (_abi.jp_loop * len(cs))(*cs)
     check(lib().jp_run_doall_spill(arr, len(cs), int(me), int(chunk), ctr.data_ptr(), _ptr(stats), int(max_ctas),
                                    _stream(stream)))
+
+
+def jp_keys_merge_p2p(peer_ptrs, keys: torch.Tensor, bar, epoch: int, err: torch.Tensor, arr=None, stream=None):
+    """peer_ptrs: every rank's key-table device pointer (ints, this rank's
+    included); bar: the shared counter (tensor or object with data_ptr())."""
+    pp = (C.c_void_p * len(peer_ptrs))(*[int(p) for p in peer_ptrs])
+    check(lib().jp_keys_merge_p2p(pp, len(peer_ptrs), keys.data_ptr(), keys.numel(), bar.data_ptr(), int(epoch),
+                                  _ptr(arr), err.data_ptr(), _stream(stream)))
 
 
 def jp_ipc_export(t: torch.Tensor) -> tuple[bytes, int]:

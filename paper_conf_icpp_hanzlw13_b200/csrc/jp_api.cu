@@ -678,6 +678,21 @@ jp_status jp_run_doall_spill(const jp_loop *views, int32_t world, int32_t me, in
   return JP_OK;
 }
 
+jp_status jp_keys_merge_p2p(const int64_t *const *peer_keys, int32_t world, int64_t *keys, int64_t len,
+                            unsigned long long *bar, int64_t epoch, void *arr, int32_t *err, jp_stream_t st) {
+  if (!peer_keys || world < 1 || world > 8 || !keys || !bar || !err || epoch < 1)
+    return fail(JP_ERR_ARG, "bad p2p merge arguments (1 <= world <= 8, epoch >= 1)");
+  if (len < 0 || len > kP2PMaxLen) return fail(JP_ERR_ARG, "p2p merge holds at most %lld slots", (long long)kP2PMaxLen);
+  for (int k = 0; k < world; k++)
+    if (!peer_keys[k]) return fail(JP_ERR_ARG, "peer key table %d is NULL", k);
+  JP_TRY(need_device());
+  JP_CUDA(launch_keys_merge_p2p(reinterpret_cast<const unsigned long long *const *>(peer_keys), world,
+                                reinterpret_cast<unsigned long long *>(keys), len, bar, (unsigned long long)epoch,
+                                static_cast<uint32_t *>(arr), err, (cudaStream_t)st),
+          "p2p key merge");
+  return JP_OK;
+}
+
 typedef int (*cu_range_fn)(unsigned long long *, size_t *, unsigned long long);
 static cu_range_fn cu_mem_range() {
   static cu_range_fn fn = nullptr;

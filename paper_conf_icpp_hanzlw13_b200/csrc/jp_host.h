@@ -62,6 +62,11 @@ cudaError_t launch_priv_stream(const Job &j, void *ws, const Layout &lo, bool cl
                                cudaStream_t st, int max_ctas = 0, bool fuse_apply = false, bool *applied = nullptr);
 cudaError_t launch_priv_finalize(const Job &j, void *ws, const Layout &lo, cudaStream_t st);
 cudaError_t launch_merge_apply(void *arr, int64_t len, const int64_t *keys, cudaStream_t st);
+// C4 over NVLink peer memory: merged max of every rank's key table (len <= kP2PMaxLen), applied to arr
+constexpr int64_t kP2PMaxLen = 16384;
+cudaError_t launch_keys_merge_p2p(const unsigned long long *const *peers, int world, unsigned long long *mine,
+                                  int64_t len, unsigned long long *bar, unsigned long long epoch, uint32_t *arr,
+                                  int *err, cudaStream_t st);
 // keys (regions 5/6) of what loop j already wrote in place (atomicMax, keys not cleared)
 cudaError_t launch_export_keys(const Job &j, void *ws, const Layout &lo, cudaStream_t st);
 // task sharing with cross-boundary spill (jp_doall.cu, C8): views[k] = rank k's affine shard

@@ -362,6 +362,86 @@ cudaError_t launch_export_keys(const Job &j, void *ws, const Layout &lo, cudaStr
   return launch_check();
 }
 
+// ---------------------------------------------------------------------------
+// C4 over NVLink peer memory (SURVEY §2c C9's role, without NCCL): one CTA per
+// rank reads every rank's key table (CUDA-IPC-mapped device pointers), keeps
+// the maximum per slot and applies it.  Two device-side barriers on a
+// monotone counter in rank 0's memory (system-scope atomics, acquire loads)
+// bracket the reads: every rank's keys are in before anyone reads (phase A),
+// and nobody clears its table for the next call before every rank has read it
+// (phase B).  epoch = 1, 2, ... per call; the counter is never reset.
+// A wait longer than ~4 s sets *err and abandons the merge (no hang).
+// ---------------------------------------------------------------------------
+constexpr int kMaxPeers = 8;
+struct PeerKeys {
+  const unsigned long long *k[kMaxPeers];
+};
+
+__device__ __forceinline__ unsigned long long ld_acquire_sys(const unsigned long long *p) {
+  unsigned long long v;
+  asm volatile("ld.acquire.sys.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+  return v;
+}
+__device__ __forceinline__ unsigned long long ld_relaxed_sys(const unsigned long long *p) {
+  unsigned long long v;
+  asm volatile("ld.relaxed.sys.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+  return v;
+}
+__device__ __forceinline__ unsigned long long gtimer() {
+  unsigned long long t;
+  asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
+  return t;
+}
+__device__ bool p2p_barrier(unsigned long long *bar, unsigned long long target, int *err) {
+  __shared__ int ok;
+  if (threadIdx.x == 0) {
+    __threadfence_system();
+    atomicAdd_system(bar, 1ull);
+    const unsigned long long t0 = gtimer();
+    ok = 1;
+    while (ld_acquire_sys(bar) < target) {
+      if (gtimer() - t0 > 4000000000ull) { ok = 0; atomicExch(err, 1); break; }
+      __nanosleep(200);
+    }
+  }
+  __syncthreads();
+  return ok;
+}
+
+__global__ void __launch_bounds__(1024) k_keys_merge_p2p(PeerKeys P, int world, unsigned long long *mine, int64_t len,
+                                                         unsigned long long *bar, unsigned long long epoch,
+                                                         uint32_t *arr, int *err) {
+  extern __shared__ unsigned long long mx[];   // len <= kP2PMaxLen
+  if (!p2p_barrier(bar, (2 * epoch - 1) * (unsigned long long)world, err)) return;
+  for (int64_t a = threadIdx.x; a < len; a += blockDim.x) {
+    unsigned long long m = 0;
+    for (int k = 0; k < world; k++) {
+      const unsigned long long v = ld_relaxed_sys(P.k[k] + a);
+      m = v > m ? v : m;
+    }
+    mx[a] = m;
+  }
+  __syncthreads();
+  if (!p2p_barrier(bar, 2 * epoch * (unsigned long long)world, err)) return;
+  for (int64_t a = threadIdx.x; a < len; a += blockDim.x) {
+    const unsigned long long m = mx[a];
+    mine[a] = m;
+    if (arr && m) arr[a] = (uint32_t)m;
+  }
+}
+
+cudaError_t launch_keys_merge_p2p(const unsigned long long *const *peers, int world, unsigned long long *mine,
+                                  int64_t len, unsigned long long *bar, unsigned long long epoch, uint32_t *arr,
+                                  int *err, cudaStream_t st) {
+  PeerKeys P;
+  for (int k = 0; k < kMaxPeers; k++) P.k[k] = k < world ? peers[k] : nullptr;
+  const size_t smem = 8 * (size_t)(len > 0 ? len : 1);
+  if (smem > 48 * 1024) cudaFuncSetAttribute(k_keys_merge_p2p, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+  k_keys_merge_p2p<<<1, 1024, smem, st>>>(P, world, mine, len, bar, epoch, arr, err);
+  note_launch();
+  return launch_check();
+}
+
 cudaError_t launch_merge_apply(void *arr, int64_t len, const int64_t *keys, cudaStream_t st) {
   apply(static_cast<uint32_t *>(arr), len, reinterpret_cast<const unsigned long long *>(keys), st);
   return launch_check();

@@ -70,6 +70,7 @@ def _region(ws: torch.Tensor, loop, name: str, dtype, engine=None):
 
 
 OWNER_MIN_LEN = 1 << 16
+P2P_MAX_LEN = 16384
 
 
 def _a2a_rows(rows, counts, group):
@@ -124,6 +125,64 @@ def owner_reduce_replicate(t, empty, group=None, engine=None) -> dict:
             "bytes_sent": (rows.numel() + world * pad.numel()) * t.element_size()}
 
 
+class P2PMerge:
+    """C4 for one small key table (<= 16384 slots) over NVLink peer memory
+    (jp_keys_merge_p2p): every rank maps every rank's table and rank 0's
+    barrier counter through CUDA IPC once; ``run`` merges (max per slot) and
+    optionally applies the keys to ``arr`` inside one single-CTA kernel per rank
+    -- no NCCL call, two device-side barriers."""
+
+    def __init__(self, table, group=None):
+        import paper_conf_icpp_hanzlw13_b200 as jp
+        self.jp, self.group, self.table = jp, group, table
+        self.world, self.rank = world_rank(group)
+        dev = table.device
+        self.bar = torch.zeros(1, dtype=torch.int64, device=dev)
+        self.err = torch.zeros(1, dtype=torch.int32, device=dev)
+        self.epoch = 0
+        self._opened = []
+        mine = (jp.jp_ipc_export(table), jp.jp_ipc_export(self.bar) if self.rank == 0 else None)
+        allinfo = [None] * self.world
+        dist.all_gather_object(allinfo, mine, group=group)
+        self.ptrs = []
+        for k, (h, _) in enumerate(allinfo):
+            if k == self.rank:
+                self.ptrs.append(table.data_ptr())
+            else:
+                p = jp.jp_ipc_import(*h)
+                self._opened.append((p, h[1]))
+                self.ptrs.append(p)
+        self.bar_ref = self.bar
+        if self.rank != 0:
+            p = jp.jp_ipc_import(*allinfo[0][1])
+            self._opened.append((p, allinfo[0][1][1]))
+            self.bar_ref = _RawPtr(p)
+        torch.cuda.synchronize()
+        dist.barrier(group=group)
+
+    def run(self, arr=None, stream=None):
+        self.epoch += 1
+        self.jp.jp_keys_merge_p2p(self.ptrs, self.table, self.bar_ref, self.epoch, self.err, arr, stream)
+
+    def ok(self) -> bool:
+        return int(self.err.item()) == 0
+
+    def close(self):
+        for p, off in self._opened:
+            self.jp.jp_ipc_close(p, off)
+        self._opened = []
+
+
+_P2P = {}
+
+
+def _p2p_for(t, group):
+    key = (t.data_ptr(), t.numel(), id(group))
+    if key not in _P2P:
+        _P2P[key] = P2PMerge(t, group)
+    return _P2P[key]
+
+
 def _reduce_tables(tabs, empty, group, exchange, jp):
     """MAX of each table across the ranks: dense all_reduce, or the owner form."""
     tabs = [t for t in tabs if t is not None]
@@ -176,11 +235,20 @@ def privatized_partitioned(loop, ws, prof, group=None, engine=None, exchange: st
     jp = _engine(engine)
     world, _ = world_rank(group)
     jp.jp_priv_stream(loop, prof, ws, clear_keys=True)
+    applied = 0
+    tabs = [(name, _region(ws, loop, name, torch.int64, jp)) for name in ("keys_A", "keys_T")]
+    tabs = [(n_, t) for n_, t in tabs if t is not None]
     if world > 1:
-        for name in ("keys_A", "keys_T"):
-            for t in _reduce_tables([_region(ws, loop, name, torch.int64, jp)], 0, group, exchange, jp):
-                owner_reduce_replicate(t, 0, group, jp)
-    jp.jp_priv_finalize(loop, ws)
+        for name, t in tabs:
+            if exchange == "p2p" and t.numel() <= P2P_MAX_LEN:
+                arr = loop.tensors["A" if name == "keys_A" else "T"]
+                _p2p_for(t, group).run(arr=arr.view(torch.int32) if arr is not None else None)
+                applied += 1
+                continue
+            for t2 in _reduce_tables([t], 0, group, "owner" if exchange == "owner" else "dense", jp):
+                owner_reduce_replicate(t2, 0, group, jp)
+    if applied < len(tabs) or not tabs:
+        jp.jp_priv_finalize(loop, ws)
 
 
 def schedule_partitioned(loop, ws, group=None, tau_high: float = 0.25, tls_window: int = 0, tls_w_max: int = 2048,
@@ -205,9 +273,9 @@ def schedule_partitioned(loop, ws, group=None, tau_high: float = 0.25, tls_windo
         res = jp.jp_schedule(loop, ws)
         res["scheme"] = "sharing"
         return res
-    if exchange not in ("dense", "owner"):
-        raise ValueError(f"exchange must be 'dense' or 'owner', not {exchange!r}")
-    prof = profile_partitioned(loop, ws, group, jp, exchange)
+    if exchange not in ("dense", "owner", "p2p"):
+        raise ValueError(f"exchange must be 'dense', 'owner' or 'p2p', not {exchange!r}")
+    prof = profile_partitioned(loop, ws, group, jp, "owner" if exchange == "owner" else "dense")
     mode = jp.jp_select_mode(loop, prof, tau_high)
     res = {"mode": mode, "mode_name": _abi.MODE_NAMES[mode], "profiled": 1, "prof": prof, "scheme": "sharing"}
     if mode in (_abi.JP_MODE_DOALL, _abi.JP_MODE_PRIVATIZED):

@@ -135,3 +135,57 @@ def test_stealing_two_ranks_one_gpu(case, exchange):
         p.join(timeout=120)
     assert [o[1] for o in out] == [True, True], out
     assert sum(o[4]["iters"] for o in out) == {"c5": 1 << 18, "c5big": 1 << 20, "c4": (1 << 18) + 64}[case]
+
+
+def _p2p_worker(rank, world, port, q):
+    sys.path[:0] = [ROOT, os.path.join(ROOT, "tests")]
+    os.environ.update(MASTER_ADDR="127.0.0.1", MASTER_PORT=str(port))
+    dist.init_process_group("gloo", rank=rank, world_size=world)
+    try:
+        import oracle as O
+        import paper_conf_icpp_hanzlw13_b200 as jp
+        from paper_conf_icpp_hanzlw13_b200 import dist as jd
+        import synth
+        from helpers import to_oracle
+        wl = synth.config4(n=(1 << 18) + 64, slots=1024)
+        _, A_exp, T_exp = O.run_seq(to_oracle(wl))
+        g = wl.to("cuda:0")
+        T0, A0 = g.T.clone(), g.A.clone()
+        full = jp.Loop.from_workload(g)
+        b, e = jd.sharing_ranges(wl.n, world)[rank]
+        loop = full.range(b, e)
+        ws = jp.workspace(loop)
+        ok = True
+        for _ in range(3):   # epochs 1..3 on the same counter and mappings
+            g.T.copy_(T0)
+            g.A.copy_(A0)
+            res = jd.schedule_partitioned(loop, ws, full_loop=full, exchange="p2p")
+            torch.cuda.synchronize()
+            ok &= g.T.cpu().numpy().tobytes() == T_exp.tobytes()
+            ok &= g.A.cpu().numpy()[b:e].tobytes() == A_exp[b:e].tobytes()
+            ok &= res["mode_name"] == "PRIVATIZED"
+        m = jd._P2P[next(iter(jd._P2P))]
+        ok &= m.ok() and m.epoch == 3
+        for m in jd._P2P.values():
+            m.close()
+        q.put((rank, bool(ok)))
+    except Exception:  # pragma: no cover
+        import traceback
+        q.put((rank, traceback.format_exc()))
+    finally:
+        dist.destroy_process_group()
+
+
+def test_p2p_key_merge_two_ranks():
+    """C4 over peer memory (jp_keys_merge_p2p through CUDA IPC, no NCCL): config 4's
+    privatized slots merged and applied in one kernel per rank, three epochs."""
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    port = _port()
+    ps = [ctx.Process(target=_p2p_worker, args=(r, 2, port, q)) for r in range(2)]
+    for p in ps:
+        p.start()
+    out = sorted(q.get(timeout=300) for _ in range(2))
+    for p in ps:
+        p.join(timeout=120)
+    assert out == [(0, True), (1, True)], out
