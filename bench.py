@@ -162,9 +162,19 @@ def oracle_baseline(sample_iters: int, max_runs: int = 5, budget_s: float = 10.0
         O.run_seq_inplace(L)
         times.append(time.perf_counter() - t0)
     t = statistics.median(times)
-    return {"value": sample_iters / t, "unit": "iter/s", "cores": 1, "kind": "oracle",
+    return {"value": sample_iters / t, "unit": "iter/s", "cores": 1, "kind": "oracle", "cpu_model": _cpu_model(),
             "sample": f"config2 SAXPY fp32, first {sample_iters} of the 2^28 iterations, jpo_run_seq on 1 host "
                       f"thread of {os.cpu_count()}, median of {len(times)} runs ({t:.3f} s each)"}
+
+
+def _cpu_model() -> str:
+    try:
+        for line in open("/proc/cpuinfo"):
+            if line.startswith("model name"):
+                return line.split(":", 1)[1].strip()
+    except OSError:
+        pass
+    return "unknown"
 
 
 def run_reference(args):
@@ -265,6 +275,22 @@ def modes_sweep(jp, dev, st):
         tls.append(row)
         del wl, ws, L, A0
     out["config3_tls"] = tls
+    # sensitivity run: dependence distances up to 2^20
+    sens = []
+    for d in (0.01, 0.10):
+        wl = synth.config3(d, delta=1 << 20, device=dev)
+        A0 = wl.A.clone()
+        L = jp.Loop.from_workload(wl)
+        ws = jp.workspace(L)
+        row = {"density": d, "delta": 1 << 20}
+        for tag, rec in (("", 0), ("restart_", 1)):
+            res, ms = timed(lambda: jp.jp_schedule(L, ws, stream=st, tls_recovery=rec), wl.A, A0)
+            row[tag + "schedule"] = {"mode": res["mode_name"], "ms": ms, "committed_per_s": wl.n / (ms * 1e-3),
+                                     "windows": res["tls"]["windows"], "violations": res["tls"]["violations"],
+                                     "recovery": ["restart", "onchip"][res["tls_recovery"]]}
+        sens.append(row)
+        del wl, ws, L, A0
+    out["config3_tls_delta_2e20"] = sens
     # config 4: privatized (profile once, then time the privatized run alone and the whole schedule)
     wl = synth.config4(device=dev)
     L = jp.Loop.from_workload(wl)
@@ -497,10 +523,26 @@ def partitioned_config5(jp, dev, st, world, rank, steps):
         barrier(world)
         if k >= 2:
             ts.append(time.perf_counter() - t0)
+    # one more call with per-phase CUDA events (not in the timing above)
+    wl.A.copy_(A0)
+    barrier(world)
+    ph = jd.schedule_stealing(full, ws, chunk_iters=65536, timings=True)["phases"]
+    phases = {k: max_over_ranks(v, world, dev) for k, v in ph.items()}
+    busy = [0.0] * world
+    if world > 1:
+        bt = torch.zeros(world, dtype=torch.float64, device=dev)
+        bt[rank] = ph["busy_ms"]
+        torch.distributed.all_reduce(bt)
+        busy = bt.tolist()
+    else:
+        busy = [ph["busy_ms"]]
+    n_stolen = res["stolen"]
     ms = max_over_ranks(statistics.median(ts) * 1e3, world, dev)
     out = {"workload": "config5 mixed ADD_C int32 N=2^24, multi-rank task stealing (chunk 2^16)", "ms": ms,
            "iters_per_s": wl.n / (ms * 1e-3), "n_tasks": res["n_tasks"], "n_batches": res["n_batches"],
-           "rank0_iters": res["rank_work"]["iters"], "tls": res["tls"],
+           "rank0_iters": res["rank_work"]["iters"], "tls": res["tls"], "phases_max_over_ranks": phases,
+           "busy_ms_per_rank": busy, "stolen_chunks": n_stolen,
+           "merge": "C4 all_reduce MAX over 2^24 int64 keys (128 MiB) + apply, per batch",
            "timing": "wall clock between barriers, max over ranks"}
     del wl, A0, full, ws
     return out

@@ -304,7 +304,7 @@ def _levels(conf, nt):
 
 
 def schedule_stealing(full, ws, group=None, chunk_iters: int = 65536, tau_high: float = 0.25, speed=None,
-                      speed_tls: float = 1.0, exchange: str = "dense", engine=None) -> dict:
+                      speed_tls: float = 1.0, exchange: str = "dense", engine=None, timings: bool = False) -> dict:
     """Task stealing of one loop across the ranks (Alg. 1; SURVEY
     Sec.8(e) "Mixed").  Every rank holds full replicas (``full``, workspace
     ``ws`` of the whole loop):
@@ -330,6 +330,14 @@ def schedule_stealing(full, ws, group=None, chunk_iters: int = 65536, tau_high: 
     world, rank = world_rank(group)
     n = full.n
     nck = -(-n // chunk_iters)
+    marks = []   # (phase, event) on the current stream when timings=True
+
+    def mark(name):
+        if timings:
+            ev = torch.cuda.Event(enable_timing=True)
+            ev.record()
+            marks.append((name, ev))
+    mark("start")
     c0, c1 = rank * nck // world, (rank + 1) * nck // world
     b, e = min(c0 * chunk_iters, n), min(c1 * chunk_iters, n)
     loop = full.range(b, e)
@@ -340,6 +348,7 @@ def schedule_stealing(full, ws, group=None, chunk_iters: int = 65536, tau_high: 
     cc[3 * c0:3 * c1] = cc_loc[:3 * (c1 - c0)]
     if world > 1:
         dist.all_reduce(cc, group=group)
+    mark("profile")
     tasks, conf = jp.jp_plan_tasks(full, cc.cpu(), chunk_iters, ws, tau_high)
     lv = _levels(conf, len(tasks))
     chunks, stolen = jp.jp_plan_stealing(tasks, world, chunk_iters, speed, speed_tls)
@@ -349,7 +358,10 @@ def schedule_stealing(full, ws, group=None, chunk_iters: int = 65536, tau_high: 
     ccl = cc.cpu().tolist()
     tls_stats = {"committed": 0, "executed": 0, "windows": 0, "violations": 0}
     mine = {"chunks": 0, "iters": 0}
+    mark("plan")
+    busy = merge = 0.0
     for level in range(max(lv) + 1 if lv else 0):
+        mark("level")
         for name in ("keys_A", "keys_T"):
             t = _region(ws, full, name, torch.int64, jp)
             if t is not None:
@@ -383,12 +395,22 @@ def schedule_stealing(full, ws, group=None, chunk_iters: int = 65536, tau_high: 
                 mine["iters"] += ce - cs
             for cs, ce in runs:
                 jp.jp_priv_stream(full.range(cs, ce), _NO_RAW, ws, clear_keys=False)
+        mark("exec")
         if world > 1:
             for name in ("keys_A", "keys_T"):
                 for t in _reduce_tables([_region(ws, full, name, torch.int64, jp)], 0, group, exchange, jp):
                     owner_reduce_replicate(t, 0, group, jp)
         jp.jp_priv_finalize(full, ws)
-    return {"scheme": "stealing", "prof": prof, "n_tasks": len(tasks), "n_batches": max(lv) + 1 if lv else 0,
+        mark("merge")
+    phases = None
+    if timings:
+        torch.cuda.synchronize()
+        phases = {"profile_ms": marks[0][1].elapsed_time(marks[1][1]), "plan_ms": marks[1][1].elapsed_time(marks[2][1])}
+        for k in range(3, len(marks), 3):   # (level, exec, merge) per batch
+            busy += marks[k][1].elapsed_time(marks[k + 1][1])
+            merge += marks[k + 1][1].elapsed_time(marks[k + 2][1])
+        phases.update(busy_ms=busy, merge_ms=merge)
+    return {"scheme": "stealing", "phases": phases, "prof": prof, "n_tasks": len(tasks), "n_batches": max(lv) + 1 if lv else 0,
             "tasks": tasks, "chunks": chunks, "stolen": stolen, "tls": tls_stats, "rank_work": mine}
 
 
