@@ -100,7 +100,13 @@ typedef struct { int64_t committed, executed, windows, violations; } jp_tls_stat
  * opcodes), 2 cooperative all-SM path (HBM stamps, software grid barrier),
  * 3 one thread-block cluster of `cluster` CTAs (HBM stamps, cluster barriers,
  * W <= 32*(144*cluster - 1)).  cluster: 1..16, 0 = auto (smallest power of two
- * >= 4 that holds the window); ignored by paths 1 and 2.                       */
+ * >= 4 that holds the window); ignored by paths 1 and 2.  path 7: no
+ * speculation -- one warp runs the loop in program order, 32 iterations per
+ * batch, in-batch RAW forwarded by shuffles in dependence order, in-batch WAW
+ * resolved to the last writer, the next batch's loads overlapped and patched
+ * (mode C, on the device; jp_serial.cu).  Its stats: committed =
+ * executed = n, windows = batches, violations = forwarded in-batch reads;
+ * window / w_max / cluster / guided / recovery are ignored.                  */
 /* Mis-speculation recovery (jp_tls_cfg.recovery).
  * JP_TLS_RESTART (reading A6): commit the prefix before the first violator and
  *   restart the next window there; windows per the policy above.
@@ -139,7 +145,9 @@ typedef struct {
                                    (measured optimum of the single-CTA path)      */
   int32_t tls_recovery;         /* 0 auto (JP_TLS_ONCHIP when the profile shows
                                    waw_iters == 0, else JP_TLS_RESTART), 1 restart,
-                                   2 on-chip                                      */
+                                   2 on-chip.  With tls_path 0 and tls_recovery 0
+                                   a SEQ_RECOMMENDED loop (mode C) runs on the
+                                   one-warp program-order path 7              */
   int32_t static_check;         /* 0: jp_static_check before profiling (affine,
                                    conflict-free loops run as DOALL unprofiled);
                                    1: skip it                                     */
@@ -157,7 +165,8 @@ typedef struct {
                                    fixed window under JP_TLS_ONCHIP                */
   int32_t tls_path;             /* TLS: jp_tls_cfg.path that ran (1, 2, 3; 4 tiny
                                    one-CTA schedule; 5 / 6 on-chip recovery on a
-                                   cluster / on every SM)                         */
+                                   cluster / on every SM; 7 one-warp program order
+                                   for mode C)                                    */
   int32_t tls_guided;           /* TLS: 1 when the guide (jp_tls_guide) steered it    */
   int32_t tls_recovery;         /* TLS: jp_tls_recovery that ran                      */
   int32_t tls_cluster;          /* TLS: CTAs of the cluster (paths 3, 5) or grid (6)  */

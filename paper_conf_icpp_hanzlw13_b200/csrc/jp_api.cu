@@ -500,6 +500,13 @@ static jp_status tls_plan(const Job &j, const jp_tls_cfg *cfg, const jp_profile 
   tp.waw = (hA || hT) && !(prof && prof->waw_iters == 0);
   const int64_t wcap = tp.window > 0 ? tp.window : tp.w_max;
   int path = cfg ? cfg->path : 0;
+  if (path == 7) {   // mode C on the device: one warp, program order (jp_serial.cu); nothing speculates
+    tp.path = 7;
+    tp.guided = false;
+    tp.recovery = JP_TLS_RESTART;
+    tp.cluster = 1;
+    return JP_OK;
+  }
   int cl = cfg ? cfg->cluster : 0;
   if (cl < 0 || cl > 16 || (cl & (cl - 1)))
     return fail(JP_ERR_ARG, "cluster must be 0 (auto) or a power of two <= 16 (got %d)", cl);
@@ -610,7 +617,9 @@ static jp_status run_tls_job(const jp_loop *L, const Job &j, const jp_tls_cfg *c
   int64_t *hdr = at<int64_t>(ws, lo, R_HEADER);
   const uint32_t *bits = tp.guided ? at<uint32_t>(ws, lo, R_GUIDE) : nullptr;
   const uint32_t *bsrc = bits ? bits + (L->n + 31) / 32 : nullptr;
-  if (tp.path == 5) {
+  if (tp.path == 7) {
+    JP_CUDA(launch_serial(j, &hdr[H_TLS_COMMITTED], st), "serial warp");
+  } else if (tp.path == 5) {
     JP_CUDA(launch_tls_fwd(j, tp.window, tp.cluster, bits, bsrc, &hdr[H_TLS_COMMITTED], st), "tls on-chip");
   } else if (tp.path == 6) {
     auto *S = at<unsigned long long>(ws, lo, R_TLS_S_A);
@@ -935,14 +944,18 @@ static jp_status run_mode(const jp_loop *L, const Job &j, int mode, const jp_pro
     // window cap from the density when not given; profile-guided mode B
     // where it helps
     // recovery: on chip (reading B7) whenever the profile allows it, unless asked otherwise
-    const int rec = c.tls_recovery == 1 ? JP_TLS_RESTART
+    // mode C (TD density above tau_high, "sequential"): the one-warp
+    // program-order path unless a TLS path or recovery was asked for
+    const bool serial = mode == JP_MODE_SEQ_RECOMMENDED && c.tls_path == 0 && c.tls_recovery == 0;
+    const int rec = serial ? JP_TLS_RESTART
+                    : c.tls_recovery == 1 ? JP_TLS_RESTART
                     : c.tls_recovery == 2 || (c.tls_path == 0 && prof && prof->waw_iters == 0) ? JP_TLS_ONCHIP
                                                                                             : JP_TLS_RESTART;
     const int64_t wm = c.tls_w_max > 0 ? c.tls_w_max : auto_w_max(prof);
-    jp_tls_cfg tc{c.tls_window, wm, c.tls_path, 0, 0, rec};
+    jp_tls_cfg tc{c.tls_window, wm, serial ? 7 : c.tls_path, 0, 0, rec};
     TlsPlan tp;
     JP_TRY(run_tls_job(L, j, &tc, prof, ws, ws_bytes, &res->tls, st, true, &tp, guide_ready));
-    res->tls_w_max = rec == JP_TLS_ONCHIP ? tp.window : wm;
+    res->tls_w_max = tp.path == 7 ? 32 : rec == JP_TLS_ONCHIP ? tp.window : wm;
     res->tls_path = tp.path;
     res->tls_guided = tp.guided ? 1 : 0;
     res->tls_recovery = rec;
@@ -1299,8 +1312,7 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
   res->mode = select_mode_counts(p.n, p.raw_iters, p.war_iters, p.waw_iters, c.tau_high);
   res->n_tasks = 1;
   res->n_batches = 1;
-  const int run = res->mode == JP_MODE_SEQ_RECOMMENDED ? JP_MODE_TLS : res->mode;
-  return run_mode(L, j, run, &p, c, ws, ws_bytes, res, st, gfuse && p.waw_iters == 0);
+  return run_mode(L, j, res->mode, &p, c, ws, ws_bytes, res, st, gfuse && p.waw_iters == 0);
 }
 
 

@@ -62,6 +62,8 @@ cudaError_t launch_priv_stream(const Job &j, void *ws, const Layout &lo, bool cl
                                cudaStream_t st, int max_ctas = 0, bool fuse_apply = false, bool *applied = nullptr);
 cudaError_t launch_priv_finalize(const Job &j, void *ws, const Layout &lo, cudaStream_t st);
 cudaError_t launch_merge_apply(void *arr, int64_t len, const int64_t *keys, cudaStream_t st);
+// mode C on the device (jp_serial.cu): one warp runs the loop in program order; stats[4] as TLS
+cudaError_t launch_serial(const Job &j, int64_t *stats, cudaStream_t st);
 // C4 over NVLink peer memory: merged max of every rank's key table (len <= kP2PMaxLen), applied to arr
 constexpr int64_t kP2PMaxLen = 16384;
 cudaError_t launch_keys_merge_p2p(const unsigned long long *const *peers, int world, unsigned long long *mine,

@@ -813,3 +813,60 @@ def test_schedule_profile_interleaved_tables(op, seed, pairs, monkeypatch):
             res["prof"]["first_raw_iter"]) == (p["raw_iters"], p["war_iters"], p["waw_iters"], p["first_raw_iter"])
     _, A, T = O.run_seq(ref)
     check_arrays(g, A, T)
+
+
+# ---------------------------------------------------------------------------
+# mode C on the device: one warp in program order (jp_tls_cfg.path 7)
+# ---------------------------------------------------------------------------
+def _chain(n, op=O.OP_ADD_C, dtype=O.I32, stride=1):
+    """Every iteration reads what iteration i - stride wrote (d_raw ~ 100%)."""
+    ar = torch.arange(n, dtype=torch.int32)
+    g = np.random.default_rng(n)
+    A = torch.from_numpy(g.integers(0, 1 << 20, size=n).astype(np.int32)) if dtype == O.I32 else \
+        torch.from_numpy(((g.integers(0, 2**23, size=n) * 2.0**-22) - 1).astype(np.float32))
+    r = torch.clamp(ar - stride, min=0)
+    if op == O.OP_STENCIL2:
+        return synth.Workload("gs", op, dtype, n, A, r=r, r2=torch.clamp(ar + 1, max=n - 1), w=ar.clone(),
+                              c0=float(np.float32(0.5)) if dtype == O.F32 else 3)
+    return synth.Workload("chain", op, dtype, n, A, r=r, w=ar.clone(), c0=7 if dtype == O.I32 else 1.1)
+
+
+@pytest.mark.parametrize("op", [O.OP_ADD_C, O.OP_SAXPY, O.OP_PRIV_TMP, O.OP_STENCIL2])
+@pytest.mark.parametrize("dtype", [O.I32, O.F32])
+@pytest.mark.parametrize("n,len_a,seed", [(1, 8, 1), (33, 16, 2), (1000, 64, 3), (5000, 4096, 4),
+                                          (70001, 3000, 5), (40000, 1 << 16, 6)])
+def test_serial_warp_matches_oracle(op, dtype, n, len_a, seed):
+    """path 7 on random loops (in-batch RAW chains, WAW, identity streams):
+    arrays equal the sequential oracle, stats count batches."""
+    wl = random_loop(seed * 13 + op * 3 + dtype, op, dtype, n, len_a=len_a)
+    ref = to_oracle(wl)
+    _, A, T = O.run_seq(ref)
+    g = gpu(wl)
+    L = jp.Loop.from_workload(g)
+    st = jp.jp_run_tls(L, path=7, ws=jp.workspace(L))
+    torch.cuda.synchronize()
+    check_arrays(g, A, T)
+    assert st["committed"] == n and st["executed"] == n and st["windows"] == -(-n // 32)
+
+
+@pytest.mark.parametrize("case", ["chain1", "chain3", "gs_f32", "gs_i32", "chain_saxpy"])
+def test_schedule_mode_c_runs_serial(case):
+    """A loop above tau_high (mode C) runs on the one-warp path through
+    jp_schedule and ends in the sequential state; larger than the tiny path."""
+    n = (1 << 16) + 17
+    wl = {"chain1": lambda: _chain(n), "chain3": lambda: _chain(n, stride=3),
+          "gs_f32": lambda: _chain(n, O.OP_STENCIL2, O.F32), "gs_i32": lambda: _chain(n, O.OP_STENCIL2, O.I32),
+          "chain_saxpy": lambda: _chain(n, O.OP_SAXPY, O.F32)}[case]()
+    if wl.op == O.OP_SAXPY:
+        wl.X = wl.A.clone()
+        wl.w = wl.r.clone()   # Y[w] = c0 X[r] + Y[w]: SAXPY reads its own write address
+    ref = to_oracle(wl)
+    _, A, T = O.run_seq(ref)
+    g = gpu(wl)
+    L = jp.Loop.from_workload(g)
+    res = jp.jp_schedule(L, jp.workspace(L))
+    torch.cuda.synchronize()
+    check_arrays(g, A, T)
+    if O.profile(ref)["raw_iters"] > 0.25 * n:
+        assert res["mode"] == jp.JP_MODE_SEQ_RECOMMENDED and res["tls_path"] == 7, res
+        assert res["task_mode_iters"][jp.JP_MODE_SEQ_RECOMMENDED] == n
