@@ -8,7 +8,9 @@
 // batches of 32 consecutive iterations, exactly in program order:
 //   * in-batch RAW: lane j's exposed A read takes the value of the LATEST
 //     earlier lane k < j that writes the same element (32 shuffle rounds find
-//     it), resolved in dependence order (one shuffle round per chain link);
+//     it), resolved in dependence order: one-source bodies (ADD_C, SAXPY) get
+//     their depth by pointer jumping and run max-depth + 1 vote-free shuffle
+//     rounds; STENCIL2 (two sources) polls readiness one round per link;
 //   * in-batch WAW: only the last writer of an element stores it
 //     (__match_any_sync groups, highest lane);
 //   * the next batch's operands (and the indices of the batch after it) are
@@ -100,7 +102,26 @@ __global__ void __launch_bounds__(32, 1) k_serial_warp(DLoop L, int64_t *stats) 
     // travels as one 64-bit word (value | done << 32)
     bool done = c.wa < 0;
     uint32_t va = 0, vt = 0;
-    if (!__all_sync(kFull, s0 < 0 && s1 < 0)) {
+    if constexpr (OP == JP_OP_ADD_C || OP == JP_OP_SAXPY) {
+      // one source per lane: its depth in the dependence forest by pointer
+      // jumping (5 rounds), then exactly max-depth + 1 value rounds, no votes
+      const int src = OP == JP_OP_ADD_C ? s0 : s1;
+      int dep = src >= 0, p = src;
+      for (int k = 0; k < 5 && __any_sync(kFull, p >= 0); k++) {
+        const int q = p < 0 ? lane : p;
+        const int pd = __shfl_sync(kFull, dep, q), pp = __shfl_sync(kFull, p, q);
+        if (p >= 0) { dep += pd; p = pp; }
+      }
+      const int maxd = (int)__reduce_max_sync(kFull, (unsigned)(done ? 0 : dep));
+      const int q = src < 0 ? lane : src;
+      for (int rd = 0; rd <= maxd; rd++) {
+        const uint32_t v = __shfl_sync(kFull, va, q);
+        if (!done && dep == rd) {
+          if (src >= 0) { if (OP == JP_OP_ADD_C) c.o0 = v; else c.o1 = v; }
+          va = ser_body<OP, DT>(L, c.o0, c.o1, vt);
+        }
+      }
+    } else if (!__all_sync(kFull, s0 < 0 && s1 < 0)) {
       for (;;) {
         const unsigned long long me = (unsigned long long)done << 32 | va;
         constexpr bool has0 = OP == JP_OP_ADD_C || OP == JP_OP_STENCIL2;   // operand 0 may be an A read
