@@ -266,8 +266,9 @@ def jp_plan_tasks(loop, chunk_counts, chunk_iters, ws, tau_high=0.25):
     for u in range(len(tasks)):
         for t in range(u):
             (wt, rt), (wu, ru) = sets[t], sets[u]
-            if wt & (wu | ru) or rt & wu:
+            if wt & (wu | ru) or rt & wu:   # symmetric, as jp.h states it
                 conf[u] |= 1 << t
+                conf[t] |= 1 << u
     return [tuple(x) for x in tasks], conf
 
 

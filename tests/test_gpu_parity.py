@@ -870,3 +870,33 @@ def test_schedule_mode_c_runs_serial(case):
     if O.profile(ref)["raw_iters"] > 0.25 * n:
         assert res["mode"] == jp.JP_MODE_SEQ_RECOMMENDED and res["tls_path"] == 7, res
         assert res["task_mode_iters"][jp.JP_MODE_SEQ_RECOMMENDED] == n
+
+
+@pytest.mark.parametrize("seed", range(6))
+def test_plan_tasks_matches_definition(seed):
+    """jp_plan_tasks (tasks = maximal same-mode chunk runs, PDG from per-address
+    task masks) against its plain definition (tests/fake_engine.py: Fig. 2(b)
+    per chunk via oracle/sched.select_mode, address sets per task, pairwise
+    intersection) on loops mixing DOALL / privatized / TLS regions."""
+    import fake_engine as fe
+    g = np.random.default_rng(seed)
+    n, chunk = 8192, 1024
+    if seed % 2:
+        wl = synth.config5(n=n, delta=64)
+    else:
+        wl = random_loop(seed, O.OP_ADD_C, O.I32, n, len_a=3 * n)
+        # perturb: some chunks independent permutations (DOALL), others dense
+        for k in range(0, n // chunk, 2):
+            perm = torch.from_numpy((g.permutation(chunk) + k * chunk).astype(np.int32))
+            wl.r[k * chunk:(k + 1) * chunk] = perm
+            wl.w[k * chunk:(k + 1) * chunk] = perm
+    gw = gpu(wl)
+    L = jp.Loop.from_workload(gw)
+    ws = jp.workspace(L)
+    cc = torch.zeros(3 * (n // chunk), dtype=torch.int64, device="cuda")
+    jp.jp_profile_density(L, ws, chunk_iters=chunk, chunk_counts=cc)
+    tasks, conf = jp.jp_plan_tasks(L, cc.cpu(), chunk, ws)
+    Lc = jp.Loop.from_workload(wl)
+    et, ec = fe.jp_plan_tasks(Lc, cc.cpu(), chunk, None)
+    assert tasks == et
+    assert conf[:len(tasks)] == ec[:len(tasks)]
