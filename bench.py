@@ -527,6 +527,19 @@ def partitioned_config5(jp, dev, st, world, rank, steps):
     wl.A.copy_(A0)
     barrier(world)
     ph = jd.schedule_stealing(full, ws, chunk_iters=65536, timings=True)["phases"]
+    # device-side stealing (jp_run_priv_claim): chunks claimed at run time
+    dts = []
+    for k in range(4):
+        wl.A.copy_(A0)
+        torch.cuda.synchronize()
+        barrier(world)
+        t0 = time.perf_counter()
+        dres = jd.schedule_stealing(full, ws, chunk_iters=65536, dynamic=True)
+        torch.cuda.synchronize()
+        barrier(world)
+        if k >= 1:
+            dts.append(time.perf_counter() - t0)
+    dyn_ms = max_over_ranks(statistics.median(dts) * 1e3, world, dev)
     phases = {k: max_over_ranks(v, world, dev) for k, v in ph.items()}
     busy = [0.0] * world
     if world > 1:
@@ -542,6 +555,8 @@ def partitioned_config5(jp, dev, st, world, rank, steps):
            "iters_per_s": wl.n / (ms * 1e-3), "n_tasks": res["n_tasks"], "n_batches": res["n_batches"],
            "rank0_iters": res["rank_work"]["iters"], "tls": res["tls"], "phases_max_over_ranks": phases,
            "busy_ms_per_rank": busy, "stolen_chunks": n_stolen,
+           "dynamic": {"ms": dyn_ms, "iters_per_s": wl.n / (dyn_ms * 1e-3), "rank0": dres["rank_work"],
+                       "what": "the batch's partitioned chunks claimed on the device (jp_run_priv_claim)"},
            "merge": "C4 all_reduce MAX over 2^24 int64 keys (128 MiB) + apply, per batch",
            "timing": "wall clock between barriers, max over ranks"}
     del wl, A0, full, ws

@@ -392,6 +392,23 @@ jp_status jp_merge_apply(void *arr, int64_t len, const int64_t *keys, jp_stream_
 jp_status jp_plan_tasks(const jp_loop *L, const int64_t *chunk_counts /* host */, int64_t chunk_iters, double tau_high,
                         void *ws, size_t ws_bytes, int64_t *tasks /* host [192] */, int32_t *n_tasks /* host */,
                         uint64_t *conf /* host [64] */, jp_stream_t st);
+/* Device-side task stealing of privatized work (Alg. 1: an idle
+ * worker steals from the queues of the others).  chunks (device [2 * m]):
+ * (start, end) local iterations of L, every chunk free of RAW (a DOALL or
+ * PRIVATIZED task's chunks); first (host [world + 1], first[0] = 0): rank k's
+ * block of the list is entries [first[k], first[k+1]).  Each rank runs the
+ * kernel on its own replica (L, ws): it claims its block's chunks ascending,
+ * then the tail of the block with the most unclaimed chunks (ties: lowest
+ * rank), with the counter protocol of jp_run_doall_spill (ctr [world] uint64
+ * visible to every rank, zero before any rank starts; each chunk runs once).
+ * A chunk runs the privatized body: exposed reads see the replica, keyed
+ * writes go to ws's key tables by atomicMax (NOT cleared; C4 merges them
+ * across ranks afterwards), identity writes are stored in place.  stats
+ * (device [3] int64, nullable, accumulated): own iterations, stolen
+ * iterations, stolen chunks.  Stream-ordered.                              */
+jp_status jp_run_priv_claim(const jp_loop *L, const int64_t *chunks, const int64_t *first /* host [world+1] */,
+                            int32_t world, int32_t me, unsigned long long *ctr, int64_t *stats, void *ws,
+                            size_t ws_bytes, int32_t max_ctas, jp_stream_t st);
 /* Packed last-writer keys (regions keys_A / keys_T of ws, NOT cleared) of what
  * loop L has already written in place: for every iteration i and every
  * indirectly written element a, keys[a] = max(keys[a], (iter_base+i+1) << 32 |

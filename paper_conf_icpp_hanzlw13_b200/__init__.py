@@ -25,7 +25,7 @@ __all__ = [
     "jp_profile_classify", "jp_profile_density", "jp_select_mode", "jp_run_doall", "jp_run_privatized",
     "jp_priv_stream", "jp_priv_finalize", "jp_doall_kernel", "jp_tls_guide", "tls_first_window", "jp_run_tls", "jp_schedule", "jp_stage_bytes", "jp_schedule_host",
     "jp_plan_sharing", "jp_plan_stealing", "jp_merge_apply",
-    "jp_plan_tasks", "jp_export_keys", "jp_keys_merge_p2p", "jp_run_doall_spill", "jp_ipc_export", "jp_ipc_import", "jp_ipc_close",
+    "jp_plan_tasks", "jp_export_keys", "jp_keys_merge_p2p", "jp_run_priv_claim", "jp_run_doall_spill", "jp_ipc_export", "jp_ipc_import", "jp_ipc_close",
     "jp_sparse_scratch_bytes", "jp_sparse_pack", "jp_sparse_reduce_max", "jp_sparse_gather", "jp_sparse_scatter",
     "jp_last_error", "jp_version", "jp_launch_count",
 ]
@@ -362,6 +362,15 @@ def jp_run_doall_spill(views, me: int, chunk: int, ctr: torch.Tensor, stats=None
     arr = (_abi.jp_loop * len(cs))(*cs)
     check(lib().jp_run_doall_spill(arr, len(cs), int(me), int(chunk), ctr.data_ptr(), _ptr(stats), int(max_ctas),
                                    _stream(stream)))
+
+
+def jp_run_priv_claim(loop: Loop, chunks: torch.Tensor, first, me: int, ctr, ws, stats=None, max_ctas: int = 0,
+                      stream=None):
+    """chunks: int64 device tensor [m, 2] of (start, end); first: world+1 ints."""
+    fl = (C.c_int64 * len(first))(*[int(x) for x in first])
+    p, nb = _ws(ws)
+    check(lib().jp_run_priv_claim(loop.ref, chunks.data_ptr() if chunks.numel() else None, fl, len(first) - 1, int(me),
+                                  ctr.data_ptr(), _ptr(stats), p, nb, int(max_ctas), _stream(stream)))
 
 
 def jp_keys_merge_p2p(peer_ptrs, keys: torch.Tensor, bar, epoch: int, err: torch.Tensor, arr=None, stream=None):

@@ -687,6 +687,25 @@ jp_status jp_run_doall_spill(const jp_loop *views, int32_t world, int32_t me, in
   return JP_OK;
 }
 
+jp_status jp_run_priv_claim(const jp_loop *L, const int64_t *chunks, const int64_t *first, int32_t world, int32_t me,
+                            unsigned long long *ctr, int64_t *stats, void *ws, size_t ws_bytes, int32_t max_ctas,
+                            jp_stream_t st) {
+  JP_TRY(check_loop(L));
+  if (!first || world < 1 || world > 8 || me < 0 || me >= world || !ctr)
+    return fail(JP_ERR_ARG, "need 1 <= world <= 8, 0 <= me < world, first[world+1] and a counter table");
+  if (first[0] != 0) return fail(JP_ERR_ARG, "first[0] must be 0");
+  for (int k = 0; k < world; k++)
+    if (first[k + 1] < first[k] || first[k + 1] - first[k] >= (1LL << 31))
+      return fail(JP_ERR_ARG, "rank blocks must be ordered and < 2^31 chunks");
+  if (first[world] > 0 && !chunks) return fail(JP_ERR_ARG, "NULL chunk list");
+  JP_TRY(need_device());
+  Layout lo;
+  JP_TRY(check_ws(L, ws, ws_bytes, JP_WS_PRIV, lo));
+  JP_CUDA(launch_priv_claim(make_job(L), ws, lo, chunks, first, world, me, ctr, stats, max_ctas, (cudaStream_t)st),
+          "priv claim");
+  return JP_OK;
+}
+
 jp_status jp_keys_merge_p2p(const int64_t *const *peer_keys, int32_t world, int64_t *keys, int64_t len,
                             unsigned long long *bar, int64_t epoch, void *arr, int32_t *err, jp_stream_t st) {
   if (!peer_keys || world < 1 || world > 8 || !keys || !bar || !err || epoch < 1)

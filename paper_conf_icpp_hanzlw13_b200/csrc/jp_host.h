@@ -64,6 +64,10 @@ cudaError_t launch_priv_finalize(const Job &j, void *ws, const Layout &lo, cudaS
 cudaError_t launch_merge_apply(void *arr, int64_t len, const int64_t *keys, cudaStream_t st);
 // mode C on the device (jp_serial.cu): one warp runs the loop in program order; stats[4] as TLS
 cudaError_t launch_serial(const Job &j, int64_t *stats, cudaStream_t st);
+// device-side task stealing of privatized chunks (Alg. 1), keys to regions 5/6
+cudaError_t launch_priv_claim(const Job &j, void *ws, const Layout &lo, const int64_t *chunks, const int64_t *first,
+                              int world, int me, unsigned long long *ctr, int64_t *stats, int max_ctas,
+                              cudaStream_t st);
 // C4 over NVLink peer memory: merged max of every rank's key table (len <= kP2PMaxLen), applied to arr
 constexpr int64_t kP2PMaxLen = 16384;
 cudaError_t launch_keys_merge_p2p(const unsigned long long *const *peers, int world, unsigned long long *mine,

@@ -18,6 +18,7 @@
 // flush then recomputes the winner's value and issues one 64-bit global
 // atomicMax per (CTA, touched slot).
 #include <cooperative_groups.h>
+#include <cstring>
 #include "jp_host.h"
 
 namespace cg = cooperative_groups;
@@ -359,6 +360,121 @@ cudaError_t launch_export_keys(const Job &j, void *ws, const Layout &lo, cudaStr
   if (j.d.n == 0) return cudaSuccess;
   JP_DISPATCH(j.op, j.dt, run_export, j.d, at<unsigned long long>(ws, lo, R_KEYS_A),
               at<unsigned long long>(ws, lo, R_KEYS_T), st);
+  return launch_check();
+}
+
+// ---------------------------------------------------------------------------
+// Task stealing on the device (Alg. 1: "steal when empty"): the
+// privatized body over a list of chunks dealt to the ranks, each rank's block
+// claimed ascending by its owner and descending by idle ranks through one
+// system-scope atomicAdd on a packed (tail << 32 | head) counter per rank
+// (the same protocol as k_doall_spill).  Every rank works on its own replica:
+// exposed reads see the replica (legal: d_raw = 0 for these chunks), keyed
+// writes go to the rank's key tables (merged afterwards by C4), identity
+// writes are stored in place (unique per iteration).
+// ---------------------------------------------------------------------------
+constexpr int kClaimRanks = 8;
+struct ClaimArgs {
+  DLoop L;
+  const int64_t *chunks;            // [2 * nchunks] local (start, end)
+  int64_t first[kClaimRanks + 1];   // rank k owns chunk entries [first[k], first[k+1])
+  unsigned long long *ctr, *kA, *kT;
+  int64_t *stats;                   // [0] own iterations, [1] stolen iterations, [2] stolen chunks
+  int world, me;
+};
+
+__device__ __forceinline__ bool claim_chunk(unsigned long long *ctr, int64_t nb, bool tail, int64_t &c) {
+  const unsigned long long old = atomicAdd_system(ctr, tail ? (1ull << 32) : 1ull);
+  const int64_t h = (uint32_t)old, t = (uint32_t)(old >> 32);
+  if (h + t >= nb) return false;
+  c = tail ? nb - 1 - t : h;
+  return true;
+}
+
+template <int OP, int DT>
+__global__ void __launch_bounds__(256) k_priv_claim(const __grid_constant__ ClaimArgs P) {
+  __shared__ int s_rank;
+  __shared__ long long s_idx;
+  const DLoop &L = P.L;
+  int64_t own = 0, stolen = 0, nst = 0;
+  bool mine = true;
+  for (;;) {
+    if (threadIdx.x == 0) {
+      int rk = -1;
+      int64_t c = 0;
+      const int64_t nbm = P.first[P.me + 1] - P.first[P.me];
+      if (mine && claim_chunk(&P.ctr[P.me], nbm, false, c)) rk = P.me;
+      else mine = false;
+      while (rk < 0) {   // the rank with the most unclaimed chunks, ties to the lowest
+        int best = -1;
+        int64_t most = 0;
+        for (int k = 0; k < P.world; k++) {
+          if (k == P.me) continue;
+          const unsigned long long v = *(volatile unsigned long long *)&P.ctr[k];
+          const int64_t left = P.first[k + 1] - P.first[k] - (int64_t)(uint32_t)v - (int64_t)(uint32_t)(v >> 32);
+          if (left > most) { most = left; best = k; }
+        }
+        if (best < 0) break;
+        if (claim_chunk(&P.ctr[best], P.first[best + 1] - P.first[best], true, c)) rk = best;
+      }
+      s_rank = rk;
+      s_idx = rk < 0 ? 0 : P.first[rk] + c;
+    }
+    __syncthreads();
+    const int rk = s_rank;
+    const int64_t ci = s_idx;
+    __syncthreads();
+    if (rk < 0) break;
+    const int64_t cs = P.chunks[2 * ci], ce = P.chunks[2 * ci + 1];
+    for (int64_t i = cs + threadIdx.x; i < ce; i += blockDim.x) {
+      uint32_t va = 0, vt = 0;
+      body_values<OP, DT>(L, i, L.A, va, vt);
+      const int64_t a = ixl(L, L.w, i);
+      if (P.kA) atomicMax(&P.kA[a], pack_key(L.base + i, va));
+      else L.A[a] = va;
+      if constexpr (OP == JP_OP_PRIV_TMP) {
+        const int64_t b = ixl(L, L.s, i);
+        if (P.kT) atomicMax(&P.kT[b], pack_key(L.base + i, vt));
+        else L.T[b] = vt;
+      }
+    }
+    if (threadIdx.x == 0) {
+      if (rk == P.me) own += ce - cs;
+      else { stolen += ce - cs; nst++; }
+    }
+  }
+  if (threadIdx.x == 0 && P.stats) {
+    if (own) atomicAdd(reinterpret_cast<unsigned long long *>(&P.stats[0]), (unsigned long long)own);
+    if (stolen) {
+      atomicAdd(reinterpret_cast<unsigned long long *>(&P.stats[1]), (unsigned long long)stolen);
+      atomicAdd(reinterpret_cast<unsigned long long *>(&P.stats[2]), (unsigned long long)nst);
+    }
+  }
+}
+
+template <int OP, int DT>
+static void run_claim(const ClaimArgs &P, int grid, cudaStream_t st) {
+  k_priv_claim<OP, DT><<<grid, 256, 0, st>>>(P);
+  note_launch();
+}
+
+cudaError_t launch_priv_claim(const Job &j, void *ws, const Layout &lo, const int64_t *chunks, const int64_t *first,
+                              int world, int me, unsigned long long *ctr, int64_t *stats, int max_ctas,
+                              cudaStream_t st) {
+  ClaimArgs P;
+  memset(&P, 0, sizeof P);
+  P.L = j.d;
+  P.chunks = chunks;
+  for (int k = 0; k <= world; k++) P.first[k] = first[k];
+  P.ctr = ctr;
+  P.kA = at<unsigned long long>(ws, lo, R_KEYS_A);
+  P.kT = j.op == JP_OP_PRIV_TMP ? at<unsigned long long>(ws, lo, R_KEYS_T) : nullptr;
+  P.stats = stats;
+  P.world = world;
+  P.me = me;
+  int grid = num_sms() * 4;
+  if (max_ctas > 0 && grid > max_ctas) grid = max_ctas;
+  JP_DISPATCH(j.op, j.dt, run_claim, P, grid, st);
   return launch_check();
 }
 

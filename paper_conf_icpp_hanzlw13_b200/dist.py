@@ -304,7 +304,8 @@ def _levels(conf, nt):
 
 
 def schedule_stealing(full, ws, group=None, chunk_iters: int = 65536, tau_high: float = 0.25, speed=None,
-                      speed_tls: float = 1.0, exchange: str = "dense", engine=None, timings: bool = False) -> dict:
+                      speed_tls: float = 1.0, exchange: str = "dense", engine=None, timings: bool = False,
+                      dynamic: bool = False) -> dict:
     """Task stealing of one loop across the ranks (Alg. 1; SURVEY
     Sec.8(e) "Mixed").  Every rank holds full replicas (``full``, workspace
     ``ws`` of the whole loop):
@@ -321,7 +322,13 @@ def schedule_stealing(full, ws, group=None, chunk_iters: int = 65536, tau_high: 
          reads see the replica, which holds every earlier batch), rank 0 the
          batch's TLS tasks in place (then jp_export_keys) -- then C4 over the
          keys (dense or owner form) and every rank applies them: every replica
-         holds the sequential result after the last batch.  Outputs written
+         holds the sequential result after the last batch.  ``dynamic``:
+         the batch's DOALL / privatized chunks are claimed on the device
+         (jp_run_priv_claim over a counter table shared through CUDA IPC):
+         every rank starts on the chunks the plan gave it and, once idle --
+         rank 0 after the pinned TLS task -- steals the tail of the most
+         loaded rank's block, so the plan's balance is corrected at run time
+         (Alg. 1's "steal when empty" on the device).  Outputs written
          through identity indices (no key table, e.g. config 4's Y) stay with
          the rank that executed the chunk, as under task sharing (``chunks``
          of the result gives the owners).
@@ -360,6 +367,8 @@ def schedule_stealing(full, ws, group=None, chunk_iters: int = 65536, tau_high: 
     mine = {"chunks": 0, "iters": 0}
     mark("plan")
     busy = merge = 0.0
+    claim = ClaimCounters(ws.device, group) if dynamic else None
+    claimed = [0, 0, 0]
     for level in range(max(lv) + 1 if lv else 0):
         mark("level")
         for name in ("keys_A", "keys_T"):
@@ -384,6 +393,8 @@ def schedule_stealing(full, ws, group=None, chunk_iters: int = 65536, tau_high: 
                     mine["chunks"] += k1 - k0
                     mine["iters"] += e2 - s
                 continue
+            if dynamic:
+                continue
             # this rank's chunks of the task, adjacent ones run as one range (one launch)
             runs = []
             for (cs, ce, cm, owner) in sorted(c for c in chunks if c[3] == rank and s <= c[0] and c[1] <= e2):
@@ -395,6 +406,20 @@ def schedule_stealing(full, ws, group=None, chunk_iters: int = 65536, tau_high: 
                 mine["iters"] += ce - cs
             for cs, ce in runs:
                 jp.jp_priv_stream(full.range(cs, ce), _NO_RAW, ws, clear_keys=False)
+        if dynamic:   # the batch's partitioned chunks, dealt by the plan, claimed on the device
+            part = [t for t, (_, _, m) in enumerate(tasks) if lv[t] == level and
+                    m not in (_abi.JP_MODE_TLS, _abi.JP_MODE_SEQ_RECOMMENDED)]
+            blocks = [[] for _ in range(world)]
+            for (cs, ce, cm, owner) in sorted(chunks):
+                if any(tasks[t][0] <= cs and ce <= tasks[t][1] for t in part):
+                    blocks[owner].append((cs, ce))
+            first = [0]
+            for b_ in blocks:
+                first.append(first[-1] + len(b_))
+            flat = [x for b_ in blocks for c_ in b_ for x in c_]
+            dch = torch.tensor(flat if flat else [0, 0], dtype=torch.int64, device=ws.device).view(-1, 2)
+            st_ = claim.run(jp, full, dch, first, ws)
+            claimed = [a + b for a, b in zip(claimed, st_)]
         mark("exec")
         if world > 1:
             for name in ("keys_A", "keys_T"):
@@ -410,12 +435,55 @@ def schedule_stealing(full, ws, group=None, chunk_iters: int = 65536, tau_high: 
             busy += marks[k][1].elapsed_time(marks[k + 1][1])
             merge += marks[k + 1][1].elapsed_time(marks[k + 2][1])
         phases.update(busy_ms=busy, merge_ms=merge)
+    if claim is not None:
+        mine = {"chunks": mine["chunks"], "iters": mine["iters"] + claimed[0] + claimed[1],
+                "own_iters": claimed[0], "stolen_iters": claimed[1], "stolen_chunks": claimed[2]}
+        claim.close()
     return {"scheme": "stealing", "phases": phases, "prof": prof, "n_tasks": len(tasks), "n_batches": max(lv) + 1 if lv else 0,
             "tasks": tasks, "chunks": chunks, "stolen": stolen, "tls": tls_stats, "rank_work": mine}
 
 
 _NO_RAW = {"n": 0, "raw_iters": 0, "war_iters": 0, "waw_iters": 0, "first_raw_iter": -1, "d_raw": 0.0, "d_war": 0.0,
            "d_waw": 0.0}
+
+
+class ClaimCounters:
+    """The per-rank chunk counters of device-side stealing (jp_run_priv_claim),
+    in rank 0's memory and mapped by every rank through CUDA IPC."""
+
+    def __init__(self, dev, group=None):
+        import paper_conf_icpp_hanzlw13_b200 as jp
+        self.jp, self.group = jp, group
+        self.world, self.rank = world_rank(group)
+        self.ctr = torch.zeros(self.world, dtype=torch.int64, device=dev)
+        self.stats = torch.zeros(3, dtype=torch.int64, device=dev)
+        self.ref, self._opened = self.ctr, None
+        if self.world > 1:
+            info = [None] * self.world
+            dist.all_gather_object(info, jp.jp_ipc_export(self.ctr) if self.rank == 0 else None, group=group)
+            if self.rank != 0:
+                p = jp.jp_ipc_import(*info[0])
+                self._opened = (p, info[0][1])
+                self.ref = _RawPtr(p)
+
+    def run(self, jp, loop, chunks, first, ws):
+        """One batch: zero the counters (rank 0), barrier, claim kernel, barrier."""
+        if self.rank == 0:
+            self.ctr.zero_()
+        self.stats.zero_()
+        if self.world > 1:
+            torch.cuda.synchronize()
+            dist.barrier(group=self.group)
+        jp.jp_run_priv_claim(loop, chunks if first[-1] else chunks[:0], first, self.rank, self.ref, ws, self.stats)
+        if self.world > 1:
+            torch.cuda.synchronize()
+            dist.barrier(group=self.group)
+        return [int(x) for x in self.stats.tolist()]
+
+    def close(self):
+        if self._opened:
+            self.jp.jp_ipc_close(*self._opened)
+            self._opened = None
 
 
 class SpillGroup:

