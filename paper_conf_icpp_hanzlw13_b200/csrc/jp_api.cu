@@ -1317,8 +1317,12 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
   const Layout lg = layout(L);
   const bool gfuse = lg.bytes[R_GUIDE] && ws && ws_bytes >= layout_end(lg, JP_WS_PROFILE | JP_WS_GUIDE | JP_WS_TLS);
   if (gfuse) {
-    JP_TRY(jp_profile_stamp(L, ws, ws_bytes, stp));
-    JP_CUDA(launch_prof_classify_guide(j, ws, lg, st), "profile classify");
+    // large A tables: stamped straight into {minW, minR} pairs (one 8-byte entry
+    // per address for the classify lookups; the separate tables stay unwritten)
+    const bool pairs = stamp_pairs_ok(j, ws, lg);
+    if (pairs) JP_CUDA(launch_prof_stamp(j, ws, lg, st, true), "profile stamp");
+    else JP_TRY(jp_profile_stamp(L, ws, ws_bytes, stp));
+    JP_CUDA(launch_prof_classify_guide(j, ws, lg, st, pairs), "profile classify");
     int64_t h[8];
     JP_CUDA(d2h_small_sync(h, at<int64_t>(ws, lg, R_HEADER), sizeof h, st), "profile D2H");
     if (h[H_BAD]) return fail(JP_ERR_INDEX, "%lld index entries are outside their arrays", (long long)h[H_BAD]);

@@ -47,12 +47,15 @@ cudaError_t launch_validate(const Job &j, int64_t *hdr, cudaStream_t st);
 // TLS guide bitmaps (region R_GUIDE: raw words then source words) from the
 // stamp tables of a profile on the same workspace; no sync.
 cudaError_t launch_tls_guide(const Job &j, void *ws, const Layout &lo, cudaStream_t st);
-cudaError_t launch_prof_stamp(const Job &j, void *ws, const Layout &lo, cudaStream_t st);
+// pairs: stamp the A tables into interleaved {minW, minR} pairs in region 7 (see stamp_pairs_ok)
+cudaError_t launch_prof_stamp(const Job &j, void *ws, const Layout &lo, cudaStream_t st, bool pairs = false);
+bool stamp_pairs_ok(const Job &j, void *ws, const Layout &lo);
 // src_bits (nullable): also the TLS guide's RAW-source words (raw_bits then holds its raw words)
 cudaError_t launch_prof_classify(const Job &j, void *ws, const Layout &lo, uint32_t *raw_bits,
                                  int64_t chunk, int64_t *chunk_counts, cudaStream_t st, uint32_t *src_bits = nullptr);
 // counts + the TLS guide bitmaps (region 13, valid when the loop writes no address twice) in one pass
-cudaError_t launch_prof_classify_guide(const Job &j, void *ws, const Layout &lo, cudaStream_t st);
+cudaError_t launch_prof_classify_guide(const Job &j, void *ws, const Layout &lo, cudaStream_t st,
+                                       bool stamped_pairs = false);
 cudaError_t launch_doall(const Job &j, cudaStream_t st, int max_ctas = 0);
 int doall_kernel_choice();
 void set_doall_kernel_choice(int v);

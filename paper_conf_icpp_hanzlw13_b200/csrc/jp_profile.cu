@@ -41,6 +41,7 @@ struct Tabs {
   // the war and waw lookups of a written address then cost one 8-byte access
   // (one DRAM burst) instead of two in separate 64 MiB tables
   const int2 *pA;
+  int as;   // element stride of wA / rA (1; 2 when they point into the pairs)
   int sA, sT;   // pre-aggregate in shared memory
   // stamp pass over an address window [lo, lo + span) only (tables larger than
   // L2 are stamped in several passes, each with an L2-resident working set);
@@ -78,14 +79,16 @@ __device__ __forceinline__ int4 idx4(const DLoop &L, const int32_t *p, int64_t i
 }
 __device__ __forceinline__ int q4(const int4 &v, int k) { return k == 0 ? v.x : k == 1 ? v.y : k == 2 ? v.z : v.w; }
 // chk: the index came from an index array (identity indices were range-checked on the host)
+// gs: element stride of the global table (2 when the A tables are stamped
+// straight into interleaved {minW, minR} pairs, jp_schedule)
 __device__ __forceinline__ void stamp32(int32_t *g, int32_t *s, int32_t a, int32_t len, int32_t e, const Tabs &t,
-                                        int &bad, bool chk = true) {
+                                        int &bad, bool chk = true, int gs = 1) {
   if (chk && (uint32_t)a >= (uint32_t)len) { bad += t.count_bad; return; }
   if ((uint32_t)a - t.lo >= t.span) return;
   if (s) {
     if (s[a] < e) atomicMax(&s[a], e);
   } else if (g) {
-    atomicMax(&g[a], e);
+    atomicMax(&g[(int64_t)a * gs], e);
   }
 }
 __device__ __forceinline__ bool earlier32(const int32_t *tab, int32_t a, int32_t len, int32_t e) {
@@ -133,13 +136,13 @@ __global__ void __launch_bounds__(256) k_prof_stamp4(DLoop L, Tabs t, int vec, i
         // identity streams (NULL arrays) were range-checked on the host and
         // reach a table only when the array is also reached through an index
         if constexpr (OP == JP_OP_ADD_C) {
-          stamp32(t.wA, sAw, a, lenA, e, t, bad, hw);
-          stamp32(t.rA, sAr, b, lenA, e, t, bad, hr);
+          stamp32(t.wA, sAw, a, lenA, e, t, bad, hw, t.as);
+          stamp32(t.rA, sAr, b, lenA, e, t, bad, hr, t.as);
         } else if constexpr (OP == JP_OP_SAXPY) {
           if (hr && (uint32_t)b >= (uint32_t)lenX) bad++;
           if (hw) {
-            stamp32(t.wA, sAw, a, lenA, e, t, bad);
-            if ((uint32_t)a < (uint32_t)lenA) stamp32(t.rA, sAr, a, lenA, e, t, bad, false);
+            stamp32(t.wA, sAw, a, lenA, e, t, bad, true, t.as);
+            if ((uint32_t)a < (uint32_t)lenA) stamp32(t.rA, sAr, a, lenA, e, t, bad, false, t.as);
           }
         } else if constexpr (OP == JP_OP_PRIV_TMP) {
           if (hr && (uint32_t)b >= (uint32_t)lenX) bad++;
@@ -151,11 +154,11 @@ __global__ void __launch_bounds__(256) k_prof_stamp4(DLoop L, Tabs t, int vec, i
               if ((uint32_t)a < (uint32_t)lenT) stamp32(t.rT, nullptr, a, lenT, e, t, bad, false);
             }
           }
-          if (hw) stamp32(t.wA, sAw, q4(vc[u], k), lenA, e, t, bad);
+          if (hw) stamp32(t.wA, sAw, q4(vc[u], k), lenA, e, t, bad, true, t.as);
         } else {
-          stamp32(t.wA, sAw, a, lenA, e, t, bad, hw);
-          stamp32(t.rA, sAr, b, lenA, e, t, bad, hr);
-          stamp32(t.rA, sAr, q4(vc[u], k), lenA, e, t, bad, h2);
+          stamp32(t.wA, sAw, a, lenA, e, t, bad, hw, t.as);
+          stamp32(t.rA, sAr, b, lenA, e, t, bad, hr, t.as);
+          stamp32(t.rA, sAr, q4(vc[u], k), lenA, e, t, bad, h2, t.as);
         }
       }
     }
@@ -203,7 +206,7 @@ __global__ void __launch_bounds__(256) k_prof_count4(DLoop L, Tabs t, int vec, i
   // the writer (local iteration) behind a raw read of address a: mark it a RAW source
   auto mark_src = [&](int32_t a) {
     if constexpr (GUIDE) {
-      const int64_t j = (int64_t)(0x7FFFFFFF - t.wA[a]) - L.base;
+      const int64_t j = (int64_t)(0x7FFFFFFF - (PAIRS ? t.pA[a].x : t.wA[a])) - L.base;
       atomicOr(&gsrc[j >> 5], 1u << (j & 31));
     }
   };
@@ -245,7 +248,7 @@ __global__ void __launch_bounds__(256) k_prof_count4(DLoop L, Tabs t, int vec, i
               war = earlier32(t.rA, a, lenA, e);
               waw = earlier32(t.wA, a, lenA, e);
             }
-            raw = b == a ? waw : earlier32(t.wA, b, lenA, e);
+            raw = b == a ? waw : PAIRS ? pair32(t.pA, b, lenA).x > e : earlier32(t.wA, b, lenA, e);
             if (raw) mark_src(b);
           } else if constexpr (OP == JP_OP_SAXPY) {
             if constexpr (PAIRS) {
@@ -271,8 +274,8 @@ __global__ void __launch_bounds__(256) k_prof_count4(DLoop L, Tabs t, int vec, i
               waw = earlier32(t.wA, a, lenA, e);
             }
             const int32_t b = q4(vb[u], k), c = q4(vc[u], k);
-            const bool r0 = b == a ? waw : earlier32(t.wA, b, lenA, e);
-            const bool r1 = c == a ? waw : c == b ? r0 : earlier32(t.wA, c, lenA, e);
+            const bool r0 = b == a ? waw : PAIRS ? pair32(t.pA, b, lenA).x > e : earlier32(t.wA, b, lenA, e);
+            const bool r1 = c == a ? waw : c == b ? r0 : PAIRS ? pair32(t.pA, c, lenA).x > e : earlier32(t.wA, c, lenA, e);
             raw = r0 || r1;
             if (r0) mark_src(q4(vb[u], k));
             if (r1) mark_src(q4(vc[u], k));
@@ -524,20 +527,44 @@ static Tabs tabs_of(const DLoop &d, void *ws, const Layout &lo) {
   t.sA = t.wA && d.lenA <= kSmemSlots;
   t.sT = t.wT && d.lenT <= kSmemSlots;
   t.pA = nullptr;
+  t.as = 1;
   return t;
 }
 
-cudaError_t launch_prof_stamp(const Job &j, void *ws, const Layout &lo, cudaStream_t st) {
+// jp_schedule may stamp the A tables straight into interleaved {minW, minR}
+// pairs held in the TLS write-log region (free until TLS, which resets it):
+// large tables only (beyond L2), both tables present, region available
+bool stamp_pairs_ok(const Job &j, void *ws, const Layout &lo) {
+  const char *e = getenv("JP_CLASSIFY_PAIRS");
+  if (e && e[0] == '0') return false;
+  return lo.bytes[R_MINW_A] && lo.bytes[R_MINR_A] && lo.bytes[R_TLS_S_A] >= 8 * (size_t)j.d.lenA &&
+         j.d.lenA >= (1 << 20) && j.d.lenA > kSmemSlots && j.op != JP_OP_PRIV_TMP &&
+         (lo.off[R_TLS_S_A] & 15) == 0 && ws;
+}
+
+cudaError_t launch_prof_stamp(const Job &j, void *ws, const Layout &lo, cudaStream_t st, bool pairs) {
   int64_t *hdr = at<int64_t>(ws, lo, R_HEADER);
   cudaMemsetAsync(hdr, 0, kHeaderBytes, st);
   cudaMemsetAsync(&hdr[H_FIRST_RAW], 0xFF, sizeof(int64_t), st);   // none (= ~0 for the u64 atomicMin)
   size_t tab_bytes = 0;
   for (int r = R_MINW_A; r <= R_MINR_T; r++) {
+    if (pairs && (r == R_MINW_A || r == R_MINR_A)) continue;
     if (lo.bytes[r]) cudaMemsetAsync(static_cast<char *>(ws) + lo.off[r], 0xFF, lo.bytes[r], st);
     tab_bytes += lo.bytes[r];
   }
+  int32_t *pw = pairs ? at<int32_t>(ws, lo, R_TLS_S_A) : nullptr;
+  if (pw) {
+    cudaMemsetAsync(pw, 0xFF, 8 * (size_t)j.d.lenA, st);
+    tab_bytes += 8 * (size_t)j.d.lenA;
+  }
   if (j.d.n == 0) return launch_check();
   Tabs t = tabs_of(j.d, ws, lo);
+  if (pw) {
+    t.wA = pw;
+    t.rA = pw + 1;
+    t.as = 2;
+    t.sA = 0;
+  }
   size_t smem = 0;
   if (t.sA) smem += (size_t)j.d.lenA * 4 * (t.rA ? 2 : 1);
   if (t.sT) smem += (size_t)j.d.lenT * 4;
@@ -609,9 +636,11 @@ static void run_classify_guide(const DLoop &d, Tabs t, uint32_t *graw, uint32_t 
     k_prof_count4<OP, false><<<g, 256, 0, st>>>(d, t, idx_vec(d), hdr, nullptr, nullptr);
   } else {
     if (t.pA) {
-      k_interleave<<<grid_for(d.lenA / 4 + 1, 256, 8), 256, 0, st>>>(t.wA, t.rA, const_cast<int2 *>(t.pA), d.lenA);
+      if (t.as == 1) {
+        k_interleave<<<grid_for(d.lenA / 4 + 1, 256, 8), 256, 0, st>>>(t.wA, t.rA, const_cast<int2 *>(t.pA), d.lenA);
+        note_launch();
+      }
       k_prof_count4<OP, true, true><<<g, 256, 0, st>>>(d, t, idx_vec(d), hdr, graw, gsrc);
-      note_launch();
     } else {
       k_prof_count4<OP, true><<<g, 256, 0, st>>>(d, t, idx_vec(d), hdr, graw, gsrc);
     }
@@ -619,7 +648,7 @@ static void run_classify_guide(const DLoop &d, Tabs t, uint32_t *graw, uint32_t 
   note_launch();
 }
 
-cudaError_t launch_prof_classify_guide(const Job &j, void *ws, const Layout &lo, cudaStream_t st) {
+cudaError_t launch_prof_classify_guide(const Job &j, void *ws, const Layout &lo, cudaStream_t st, bool stamped_pairs) {
   int64_t *hdr = at<int64_t>(ws, lo, R_HEADER);
   uint32_t *bits = at<uint32_t>(ws, lo, R_GUIDE);
   if (!bits) return launch_prof_classify(j, ws, lo, nullptr, 0, nullptr, st);
@@ -633,9 +662,15 @@ cudaError_t launch_prof_classify_guide(const Job &j, void *ws, const Layout &lo,
   // until TLS runs: it holds the interleaved A tables for this pass when the
   // tables are large (beyond L2, where the second table's lookup is a DRAM burst)
   unsigned long long *scratch = at<unsigned long long>(ws, lo, R_TLS_S_A);
-  if (scratch && t.wA && t.rA && !t.sA && j.d.lenA >= (1 << 20) && ((uintptr_t)t.wA & 15) == 0 &&
-      ((uintptr_t)t.rA & 15) == 0 && getenv_int("JP_CLASSIFY_PAIRS", 1))
+  if (stamped_pairs) {   // the stamp pass wrote the pairs: no interleave pass
     t.pA = reinterpret_cast<const int2 *>(scratch);
+    t.wA = reinterpret_cast<int32_t *>(scratch);
+    t.rA = t.wA + 1;
+    t.as = 2;
+  } else if (scratch && t.wA && t.rA && !t.sA && j.d.lenA >= (1 << 20) && ((uintptr_t)t.wA & 15) == 0 &&
+             ((uintptr_t)t.rA & 15) == 0 && getenv_int("JP_CLASSIFY_PAIRS", 1)) {
+    t.pA = reinterpret_cast<const int2 *>(scratch);
+  }
   JP_DISPATCH(j.op, j.dt, run_classify_guide, j.d, t, bits, bits + nw, hdr, st);
   return launch_check();
 }
