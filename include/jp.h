@@ -307,7 +307,12 @@ jp_status jp_run_tls(const jp_loop *L, const jp_tls_cfg *cfg /* host */, const j
  * tasks (Alg. 1 P:L426-437 job pool); tasks that touch a common address with a
  * write are ordered (PDG reading A19), conflict-free tasks of one topological
  * batch run concurrently on separate streams (the TLS task on one SM, the
- * partitioned tasks on the rest).  syncs.                                     */
+ * partitioned tasks on the rest).  A SEQ_RECOMMENDED loop (mode C) runs on
+ * the one-warp program-order path 7 unless cfg asks for a TLS path or
+ * recovery.  The workspace is scratch for the whole call: the profile tables
+ * of large loops are kept interleaved in the TLS region and the minW / minR
+ * regions are not left filled (call jp_profile_density for the tables).
+ * syncs.                                                                     */
 jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfg /* host */, void *ws,
                       size_t ws_bytes, jp_sched_result *res /* host */, jp_stream_t st);
 /* Same, with every array pointer of L_host on the HOST (pinned for speed): the
