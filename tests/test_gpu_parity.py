@@ -847,6 +847,16 @@ def test_serial_warp_matches_oracle(op, dtype, n, len_a, seed):
     torch.cuda.synchronize()
     check_arrays(g, A, T)
     assert st["committed"] == n and st["executed"] == n and st["windows"] == -(-n // 32)
+    # violations = iterations whose exposed A read was written earlier in the same 32-iteration batch
+    ix = lambda a: np.arange(n) if a is None else a.numpy().astype(np.int64)  # noqa: E731
+    w = ix(wl.w)
+    reads = {O.OP_ADD_C: [ix(wl.r)], O.OP_SAXPY: [w], O.OP_PRIV_TMP: [],
+             O.OP_STENCIL2: [ix(wl.r), ix(wl.r2)]}[op]
+    fwd = 0
+    for i in range(n):
+        b0 = i - i % 32
+        fwd += any(np.any(w[b0:i] == rd[i]) for rd in reads)
+    assert st["violations"] == fwd
 
 
 @pytest.mark.parametrize("case", ["chain1", "chain3", "gs_f32", "gs_i32", "chain_saxpy"])
