@@ -317,7 +317,11 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfg /* host */, void
                       size_t ws_bytes, jp_sched_result *res /* host */, jp_stream_t st);
 /* Same, with every array pointer of L_host on the HOST (pinned for speed): the
  * arrays are copied into `stage` (device, >= jp_stage_bytes), scheduled, and
- * the written arrays copied back.  syncs.                                      */
+ * the written arrays copied back.  A determined-DOALL loop (every index NULL,
+ * ident_off 0, arrays of n elements) is pipelined instead: chunks of 2^23
+ * iterations (env JP_STAGE_CHUNK) go H2D -> kernel -> D2H on three streams, so
+ * uploads, kernels and downloads of different chunks overlap (P:L345-349,
+ * data staged "asynchronously with the kernel execution"; ws unused).  syncs. */
 size_t jp_stage_bytes(const jp_loop *L_host /* host */);
 jp_status jp_schedule_host(const jp_loop *L_host /* host */, const jp_sched_cfg *cfg,
                            void *stage, size_t stage_bytes, void *ws, size_t ws_bytes,

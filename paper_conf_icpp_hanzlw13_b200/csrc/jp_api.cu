@@ -1475,6 +1475,67 @@ size_t jp_stage_bytes(const jp_loop *L) {
   return stage_layout(L).total;
 }
 
+// Determined-DOALL loops (every index NULL, identity from element 0; mode A,
+// P:L361-362) need no profile, so staging can overlap execution chunk by chunk
+// (data "moved to the GPU in advance and asynchronously with the
+// kernel execution"): chunk c's H2D, kernel and D2H run on pool stream c % 3,
+// so one chunk's upload, another's kernel and a third's download proceed
+// together on the two copy engines and the SMs.
+static jp_status schedule_host_pipelined(const jp_loop *Lh, const Stage &sl, char *b, jp_sched_result *res,
+                                         cudaStream_t st) {
+  const int64_t n = Lh->n;
+  int64_t chunk = 1 << 23;   // measured: 2^20 5.3, 2^21 5.9, 2^22 6.15, 2^23 6.28, 2^24 6.29 G iter/s (config 2 e2e)
+  if (const char *e = getenv("JP_STAGE_CHUNK")) chunk = std::max<int64_t>(1024, atoll(e));
+  chunk = (chunk + 3) & ~(int64_t)3;
+  const bool usesX = Lh->op == JP_OP_SAXPY || Lh->op == JP_OP_PRIV_TMP;
+  const bool hasT = Lh->op == JP_OP_PRIV_TMP;
+  const bool readsA = Lh->op != JP_OP_PRIV_TMP;
+  char *dA = b + sl.off[4], *dX = usesX ? b + sl.off[5] : nullptr, *dT = hasT ? b + sl.off[6] : nullptr;
+  cudaEvent_t e0;
+  JP_CUDA(cudaEventCreateWithFlags(&e0, cudaEventDisableTiming), "event");
+  cudaEventRecord(e0, st);
+  constexpr int kPipe = 3;
+  cudaStream_t ps[kPipe];
+  for (int k = 0; k < kPipe; k++) {
+    ps[k] = g_pool.get(32 + k);
+    cudaStreamWaitEvent(ps[k], e0, 0);
+  }
+  for (int64_t c0 = 0, c = 0; c0 < n; c0 += chunk, c++) {
+    const int64_t m = std::min(chunk, n - c0);
+    cudaStream_t s = ps[c % kPipe];
+    const size_t off = 4 * (size_t)c0, nb = 4 * (size_t)m;
+    if (readsA) JP_CUDA(cudaMemcpyAsync(dA + off, static_cast<const char *>(Lh->A) + off, nb, cudaMemcpyHostToDevice, s), "H2D");
+    if (usesX) JP_CUDA(cudaMemcpyAsync(dX + off, static_cast<const char *>(Lh->X) + off, nb, cudaMemcpyHostToDevice, s), "H2D");
+    jp_loop sub = *Lh;
+    sub.n = m;
+    sub.iter_base = Lh->iter_base + c0;
+    sub.A = dA + off;
+    sub.len_A = m;
+    sub.X = dX ? dX + off : nullptr;
+    sub.len_X = dX ? m : 0;
+    sub.T = dT ? dT + off : nullptr;
+    sub.len_T = dT ? m : 0;
+    JP_CUDA(launch_doall(make_job(&sub), s), "doall chunk");
+    JP_CUDA(cudaMemcpyAsync(static_cast<char *>(Lh->A) + off, dA + off, nb, cudaMemcpyDeviceToHost, s), "D2H");
+    if (hasT) JP_CUDA(cudaMemcpyAsync(static_cast<char *>(Lh->T) + off, dT + off, nb, cudaMemcpyDeviceToHost, s), "D2H");
+  }
+  for (int k = 0; k < kPipe; k++) {
+    cudaEvent_t e;
+    cudaEventCreateWithFlags(&e, cudaEventDisableTiming);
+    cudaEventRecord(e, ps[k]);
+    cudaStreamWaitEvent(st, e, 0);
+    cudaEventDestroy(e);
+  }
+  cudaEventDestroy(e0);
+  JP_CUDA(cudaStreamSynchronize(st), "stage sync");
+  res->mode = JP_MODE_DOALL;
+  res->profiled = 0;
+  res->n_tasks = 1;
+  res->n_batches = 1;
+  res->task_mode_iters[JP_MODE_DOALL] = n;
+  return JP_OK;
+}
+
 jp_status jp_schedule_host(const jp_loop *Lh, const jp_sched_cfg *cfg, void *stage, size_t stage_bytes, void *ws,
                            size_t ws_bytes, jp_sched_result *res, jp_stream_t stp) {
   JP_TRY(check_loop(Lh));
@@ -1482,6 +1543,12 @@ jp_status jp_schedule_host(const jp_loop *Lh, const jp_sched_cfg *cfg, void *sta
   Stage sl = stage_layout(Lh);
   if (!stage || stage_bytes < sl.total) return fail(JP_ERR_WORKSPACE, "stage buffer needs %zu bytes", sl.total);
   cudaStream_t st = (cudaStream_t)stp;
+  if (!Lh->r && !Lh->r2 && !Lh->w && !Lh->s && Lh->ident_off == 0 && res && Lh->n > 0 &&
+      Lh->len_A == Lh->n && (!(Lh->op == JP_OP_SAXPY || Lh->op == JP_OP_PRIV_TMP) || Lh->len_X == Lh->n) &&
+      (Lh->op != JP_OP_PRIV_TMP || Lh->len_T == Lh->n) && !(getenv("JP_STAGE_PIPELINE") && getenv("JP_STAGE_PIPELINE")[0] == '0')) {
+    memset(res, 0, sizeof *res);
+    return schedule_host_pipelined(Lh, sl, static_cast<char *>(stage), res, st);
+  }
   jp_loop Ld = *Lh;
   char *b = static_cast<char *>(stage);
   const void *src[7] = {Lh->r, Lh->r2, Lh->w, Lh->s, Lh->A, Lh->X, Lh->T};

@@ -910,3 +910,29 @@ def test_plan_tasks_matches_definition(seed):
     et, ec = fe.jp_plan_tasks(Lc, cc.cpu(), chunk, None)
     assert tasks == et
     assert conf[:len(tasks)] == ec[:len(tasks)]
+
+
+@pytest.mark.parametrize("op,dtype", [(O.OP_SAXPY, O.F32), (O.OP_ADD_C, O.I32), (O.OP_PRIV_TMP, O.F32),
+                                      (O.OP_STENCIL2, O.F32)])
+@pytest.mark.parametrize("n,chunk", [((1 << 22) * 3 + 77, None), (10000, "1024"), (5, "1024")])
+def test_schedule_host_pipelined_doall(op, dtype, n, chunk, monkeypatch):
+    """Determined-DOALL loops through jp_schedule_host: chunked H2D / kernel /
+    D2H on three streams (pre-staging overlapped with execution)
+    gives the sequential result, ragged last chunk included."""
+    if chunk:
+        monkeypatch.setenv("JP_STAGE_CHUNK", chunk)
+    g = np.random.default_rng(n + op)
+    el = np.int32 if dtype == O.I32 else np.float32
+    mk = lambda: torch.from_numpy((g.integers(-9, 9, size=n) if dtype == O.I32  # noqa: E731
+                                   else g.standard_normal(n)).astype(el))
+    wl = synth.Workload("aff", op, dtype, n, mk(), X=mk() if op in (O.OP_SAXPY, O.OP_PRIV_TMP) else None,
+                        T=mk() if op == O.OP_PRIV_TMP else None, c0=3 if dtype == O.I32 else 1.1, c1=0.3)
+    _, A, T = O.run_seq(to_oracle(wl))
+    h = {k: v.pin_memory() for k, v in wl.arrays().items()}
+    L = jp.Loop(op, dtype, n, h["A"], X=h.get("X"), T=h.get("T"), c0=wl.c0, c1=wl.c1)
+    stage = torch.empty(jp.jp_stage_bytes(L), dtype=torch.uint8, device=DEV)
+    res = jp.jp_schedule_host(L, stage, None)
+    assert res["mode"] == jp.JP_MODE_DOALL and res["profiled"] == 0
+    assert h["A"].numpy().tobytes() == A.tobytes()
+    if T is not None:
+        assert h["T"].numpy().tobytes() == T.tobytes()
