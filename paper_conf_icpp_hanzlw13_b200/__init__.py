@@ -9,6 +9,7 @@ process groups -- every step of the loop runs in the CUDA kernels.
 from __future__ import annotations
 
 import ctypes as C
+import struct
 
 import torch
 
@@ -37,11 +38,19 @@ def _ptr(t):
     return None if t is None else t.data_ptr()
 
 
+_HAS_CUDA = None
+
+
 def _stream(stream=None):
+    """cudaStream_t of `stream`, else torch's current stream (raw accessor: the
+    tiny-loop path is launch-latency bound, config 1)."""
+    global _HAS_CUDA
     if stream is not None:
         return stream.cuda_stream if hasattr(stream, "cuda_stream") else int(stream)
-    if torch.cuda.is_available():
-        return torch.cuda.current_stream().cuda_stream
+    if _HAS_CUDA is None:
+        _HAS_CUDA = torch.cuda.is_available()
+    if _HAS_CUDA:
+        return torch._C._cuda_getCurrentRawStream(torch._C._cuda_getDevice())
     return None
 
 
@@ -253,12 +262,20 @@ def sched_cfg(scheme=JP_SCHED_SHARING, tau_high=0.25, chunk_iters=65536, tls_win
                              int(tls_w_max), int(tls_recovery), int(static_check))
 
 
+# jp_sched_result unpacked in one call (field order and natural alignment of jp.h)
+_RES_FMT = struct.Struct("=ii5q3d4qqq4qq4i")
+assert _RES_FMT.size == C.sizeof(_abi.jp_sched_result)
+
+
 def _res_dict(r: _abi.jp_sched_result) -> dict:
-    return {"mode": r.mode, "mode_name": MODE_NAMES.get(r.mode, "?"), "profiled": r.profiled,
-            "prof": _prof_dict(r.prof), "tls": {k: getattr(r.tls, k) for k, _ in _abi.jp_tls_stats._fields_},
-            "n_tasks": r.n_tasks, "n_batches": r.n_batches, "task_mode_iters": list(r.task_mode_iters),
-            "tls_w_max": r.tls_w_max, "tls_path": r.tls_path, "tls_guided": r.tls_guided,
-            "tls_recovery": r.tls_recovery, "tls_cluster": r.tls_cluster}
+    (mode, profiled, n, raw, war, waw, first, d_raw, d_war, d_waw, com, exe, win, vio, n_tasks, n_batches,
+     m0, m1, m2, m3, wmax, path, guided, rec, cl) = _RES_FMT.unpack(bytes(r))
+    return {"mode": mode, "mode_name": MODE_NAMES.get(mode, "?"), "profiled": profiled,
+            "prof": {"n": n, "raw_iters": raw, "war_iters": war, "waw_iters": waw, "first_raw_iter": first,
+                     "d_raw": d_raw, "d_war": d_war, "d_waw": d_waw},
+            "tls": {"committed": com, "executed": exe, "windows": win, "violations": vio},
+            "n_tasks": n_tasks, "n_batches": n_batches, "task_mode_iters": [m0, m1, m2, m3],
+            "tls_w_max": wmax, "tls_path": path, "tls_guided": guided, "tls_recovery": rec, "tls_cluster": cl}
 
 
 def jp_schedule(loop: Loop, ws=None, cfg=None, stream=None, **kw) -> dict:

@@ -105,8 +105,9 @@ bool affine_conflict(int64_t af, int64_t bf, int64_t ag, int64_t bg, int64_t n);
 
 // tiny loops (jp_tiny.cu): the whole schedule in one CTA's shared memory
 bool tiny_eligible(const jp_loop *L);
+// mirror (nullable, mapped pinned host [17]): header words 0..15 then seq, written by the kernel
 cudaError_t launch_tiny(const Job &j, const jp_loop *L, double tau, int64_t window, int64_t w_max, int recovery,
-                        int64_t *hdr, cudaStream_t st);
+                        int64_t *hdr, cudaStream_t st, int64_t *mirror = nullptr, unsigned long long seq = 0);
 
 struct TlsPlan {
   int64_t window, w_max, prof_raw;  // prof_raw < 0: no profile

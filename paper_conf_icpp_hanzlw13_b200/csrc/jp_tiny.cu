@@ -19,14 +19,30 @@
 
 namespace jp {
 
-constexpr int kTinyThreads = 256, kTinyK = 16;   // n <= 4096 (few warps: everything is in shared memory)
+constexpr int kTinyThreads = 1024, kTinyK = 4;   // n <= 4096 (few warps: everything is in shared memory)
 constexpr uint32_t kTinyEpochs = 0xFFFFF;        // 20-bit window counter (windows <= n <= 4096)
 
 struct TinyArgs {
   double tau;
   int64_t window, w_max;   // w_max 0: from the profiled density (as jp_schedule)
   int recovery;            // jp_sched_cfg.tls_recovery: 0 auto (on chip when no address is written twice), 1 restart
+  int64_t *mirror;         // nullable: mapped pinned host words [17] = header words 0..15, then seq
+  unsigned long long seq;
 };
+
+// the result words straight into mapped host memory, then the sequence flag:
+// the host polls the flag instead of enqueueing a D2H copy (config 1 is
+// launch-latency bound).  Every thread's stores are fenced before the flag.
+__device__ __forceinline__ void tiny_publish(const int64_t *hdr, const TinyArgs &a) {
+  if (!a.mirror) return;
+  __threadfence();
+  JP_CTA_SYNC();
+  if (threadIdx.x == 0) {
+    for (int k = 0; k < 16; k++) a.mirror[k] = hdr[k];
+    __threadfence_system();
+    *(volatile unsigned long long *)&a.mirror[16] = a.seq;
+  }
+}
 
 template <int OP> __host__ __device__ constexpr int tiny_streams() { return (OP == JP_OP_PRIV_TMP || OP == JP_OP_STENCIL2) ? 3 : 2; }
 // exposed reads of A (X is never written, T reads are covered)
@@ -111,6 +127,7 @@ __global__ void __launch_bounds__(kTinyThreads, 1) k_tiny(DLoop L, TinyArgs a, i
   JP_CTA_SYNC();
   if (s_cnt[3]) {   // JP_ERR_INDEX: nothing modified
     if (tid == 0) { hdr[H_BAD] = s_cnt[3]; hdr[H_TINY_MODE] = -1; }
+    tiny_publish(hdr, a);
     return;
   }
   // ---- classify (P2) ----
@@ -396,6 +413,7 @@ __global__ void __launch_bounds__(kTinyThreads, 1) k_tiny(DLoop L, TinyArgs a, i
     hdr[H_TINY_WMAX] = wmax_used;
     hdr[H_TINY_REC] = onchip ? JP_TLS_ONCHIP : JP_TLS_RESTART;
   }
+  tiny_publish(hdr, a);
 }
 
 size_t tiny_smem_bytes(const jp_loop *L) {
@@ -431,12 +449,14 @@ static void run_tiny_v(cudaError_t &e, const DLoop &d, TinyArgs a, size_t smem, 
 }
 
 cudaError_t launch_tiny(const Job &j, const jp_loop *L, double tau, int64_t window, int64_t w_max, int recovery,
-                        int64_t *hdr, cudaStream_t st) {
+                        int64_t *hdr, cudaStream_t st, int64_t *mirror, unsigned long long seq) {
   TinyArgs a;
   a.tau = tau;
   a.window = window;
   a.w_max = w_max;
   a.recovery = recovery;
+  a.mirror = mirror;
+  a.seq = seq;
   cudaError_t e = cudaSuccess;
   JP_DISPATCH(j.op, j.dt, run_tiny_v, e, j.d, a, tiny_smem_bytes(L), hdr, st);
   return e;
