@@ -315,18 +315,18 @@ def modes_sweep(jp, dev, st):
         wl = synth.config1(d, device=dev)
         L = jp.Loop.from_workload(wl)
         ws = jp.workspace(L)
-        res = jp.jp_schedule(L, ws, stream=st)
-        ts = []
         for _ in range(20):
+            res = jp.jp_schedule(L, ws, stream=st)
+        ts = []
+        for _ in range(200):   # jp_schedule syncs its stream: the call's wall time is the latency
             t0 = time.perf_counter()
             jp.jp_schedule(L, ws, stream=st)
-            torch.cuda.synchronize()
             ts.append(time.perf_counter() - t0)
         # the CPU oracle on the same loop (sequential run, one host thread) for context
         import oracle as O
         ref = O.Loop(wl.op, wl.dtype, wl.n, wl.A.cpu().numpy(), r=wl.r.cpu().numpy(), w=wl.w.cpu().numpy(), c0=wl.c0)
         to = []
-        for _ in range(20):
+        for _ in range(200):
             t0 = time.perf_counter()
             O.run_seq_inplace(ref)
             to.append(time.perf_counter() - t0)
