@@ -410,7 +410,8 @@ def partitioned_config4(jp, dev, st, world, rank, steps):
     prof_ms = timed(lambda: prof.update(jd.profile_partitioned(loop, ws)), steps)
     mode = jp.jp_select_mode(loop, prof, 0.25)
     ms = timed(lambda: jd.privatized_partitioned(loop, ws, prof), steps)
-    ms_p2p = timed(lambda: jd.privatized_partitioned(loop, ws, prof, exchange="p2p"), steps) if world > 1 else None
+    ms_p2p = timed(lambda: jd.privatized_partitioned(loop, ws, prof, exchange="p2p"), steps) \
+        if world > 1 and IPC_ROWS else None
     hbm, _ = peaks()
     return {"workload": "config4: PRIV_TMP fp32 N=2^26 S=1024, task sharing; step = privatized stream + C4 + finalize",
             "n": wl.n, "n_per_rank": e - b, "mode": jp.MODE_NAMES[mode], "ms": ms, "iters_per_s": wl.n / (ms * 1e-3),
@@ -529,7 +530,7 @@ def partitioned_config5(jp, dev, st, world, rank, steps):
     ph = jd.schedule_stealing(full, ws, chunk_iters=65536, timings=True)["phases"]
     # device-side stealing (jp_run_priv_claim): chunks claimed at run time
     dts = []
-    for k in range(4):
+    for k in range(4 if world == 1 or IPC_ROWS else 0):
         wl.A.copy_(A0)
         torch.cuda.synchronize()
         barrier(world)
@@ -539,7 +540,9 @@ def partitioned_config5(jp, dev, st, world, rank, steps):
         barrier(world)
         if k >= 1:
             dts.append(time.perf_counter() - t0)
-    dyn_ms = max_over_ranks(statistics.median(dts) * 1e3, world, dev)
+    dyn_ms = max_over_ranks(statistics.median(dts) * 1e3, world, dev) if dts else None
+    if not dts:
+        dres = {"rank_work": "skipped: CUDA-IPC rows at N > 1 need JP_BENCH_IPC=1"}
     phases = {k: max_over_ranks(v, world, dev) for k, v in ph.items()}
     busy = [0.0] * world
     if world > 1:
@@ -555,7 +558,8 @@ def partitioned_config5(jp, dev, st, world, rank, steps):
            "iters_per_s": wl.n / (ms * 1e-3), "n_tasks": res["n_tasks"], "n_batches": res["n_batches"],
            "rank0_iters": res["rank_work"]["iters"], "tls": res["tls"], "phases_max_over_ranks": phases,
            "busy_ms_per_rank": busy, "stolen_chunks": n_stolen,
-           "dynamic": {"ms": dyn_ms, "iters_per_s": wl.n / (dyn_ms * 1e-3), "rank0": dres["rank_work"],
+           "dynamic": {"ms": dyn_ms, "iters_per_s": wl.n / (dyn_ms * 1e-3) if dyn_ms else None,
+                       "rank0": dres["rank_work"],
                        "what": "the batch's partitioned chunks claimed on the device (jp_run_priv_claim)"},
            "merge": "C4 all_reduce MAX over 2^24 int64 keys (128 MiB) + apply, per batch",
            "timing": "wall clock between barriers, max over ranks"}
@@ -607,6 +611,12 @@ def exchange_cost(jp, dev, st):
     del wl, full, loop, ws, W, R, rows, R2
     torch.cuda.empty_cache()
     return out
+
+
+# Rows that map peer memory through CUDA IPC (spill, p2p C4, device-side
+# stealing) are tested with two ranks sharing one GPU only; on a multi-GPU box
+# they run when JP_BENCH_IPC=1 so that the default scaling run cannot stall on them.
+IPC_ROWS = os.environ.get("JP_BENCH_IPC", "0") == "1"
 
 
 def run_jp(args):
@@ -697,7 +707,8 @@ def run_jp(args):
         torch.cuda.empty_cache()
         part = partitioned_config4(jp, dev, st, world, rank, 5)
         torch.cuda.empty_cache()
-        spill = partitioned_spill(jp, dev, st, world, rank, 5)
+        spill = partitioned_spill(jp, dev, st, world, rank, 5) if world == 1 or IPC_ROWS else \
+            {"skipped": "CUDA-IPC rows at N > 1 need JP_BENCH_IPC=1"}
         torch.cuda.empty_cache()
         steal = partitioned_config5(jp, dev, st, world, rank, 3)
         torch.cuda.empty_cache()
