@@ -626,7 +626,7 @@ static int64_t auto_w_max(const jp_profile *p) {
 // workspace allow it (jp_schedule)
 static jp_status run_tls_job(const jp_loop *L, const Job &j, const jp_tls_cfg *cfg, const jp_profile *prof, void *ws,
                              size_t ws_bytes, jp_tls_stats *stats, cudaStream_t st, bool auto_guide = false,
-                             TlsPlan *plan_out = nullptr, bool guide_ready = false) {
+                             TlsPlan *plan_out = nullptr, bool guide_ready = false, bool s_clean = false) {
   TlsPlan tp;
   JP_TRY(tls_plan(j, cfg, prof, tp));
   const bool helps = tp.path == 3 || tp.path >= 5 || (tp.path == 1 && prof && prof->n > 0 && prof->raw_iters * 50 <= prof->n);
@@ -655,7 +655,7 @@ static jp_status run_tls_job(const jp_loop *L, const Job &j, const jp_tls_cfg *c
     auto *V = at<unsigned long long>(ws, lo, R_TLS_C_A);
     const int64_t lenS = S && V ? L->len_A : 0;
     JP_CUDA(launch_tls_fwd_grid(j, tp.window, bits, bsrc, S, V, lenS, reinterpret_cast<unsigned *>(&hdr[H_BAR_COUNT]),
-                                &hdr[H_TLS_COMMITTED], st),
+                                &hdr[H_TLS_COMMITTED], st, s_clean),
             "tls on-chip grid");
   } else {
     JP_CUDA(launch_tls(j, ws, lo, tp, &hdr[H_TLS_COMMITTED], st), "tls");
@@ -979,7 +979,8 @@ static Job sub_job(const Job &j, int64_t s, int64_t e) {
 }
 
 static jp_status run_mode(const jp_loop *L, const Job &j, int mode, const jp_profile *prof, const jp_sched_cfg &c,
-                          void *ws, size_t ws_bytes, jp_sched_result *res, cudaStream_t st, bool guide_ready = false) {
+                          void *ws, size_t ws_bytes, jp_sched_result *res, cudaStream_t st, bool guide_ready = false,
+                          bool s_clean = false) {
   Layout lo = layout(L);
   if (mode == JP_MODE_DOALL) {
     JP_CUDA(launch_doall(j, st), "doall");
@@ -1002,7 +1003,7 @@ static jp_status run_mode(const jp_loop *L, const Job &j, int mode, const jp_pro
     const int64_t wm = c.tls_w_max > 0 ? c.tls_w_max : auto_w_max(prof);
     jp_tls_cfg tc{c.tls_window, wm, serial ? 7 : c.tls_path, 0, 0, rec};
     TlsPlan tp;
-    JP_TRY(run_tls_job(L, j, &tc, prof, ws, ws_bytes, &res->tls, st, true, &tp, guide_ready));
+    JP_TRY(run_tls_job(L, j, &tc, prof, ws, ws_bytes, &res->tls, st, true, &tp, guide_ready, s_clean));
     res->tls_w_max = tp.path == 7 ? 32 : rec == JP_TLS_ONCHIP ? tp.window : wm;
     res->tls_path = tp.path;
     res->tls_guided = tp.guided ? 1 : 0;
@@ -1361,10 +1362,11 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
   // (A read through an index, workspace with the guide region): no separate guide pass
   const Layout lg = layout(L);
   const bool gfuse = lg.bytes[R_GUIDE] && ws && ws_bytes >= layout_end(lg, JP_WS_PROFILE | JP_WS_GUIDE | JP_WS_TLS);
+  bool pairs = false;
   if (gfuse) {
     // large A tables: stamped straight into {minW, minR} pairs (one 8-byte entry
     // per address for the classify lookups; the separate tables stay unwritten)
-    const bool pairs = stamp_pairs_ok(j, ws, lg);
+    pairs = stamp_pairs_ok(j, ws, lg);
     if (pairs) JP_CUDA(launch_prof_stamp(j, ws, lg, st, true), "profile stamp");
     else JP_TRY(jp_profile_stamp(L, ws, ws_bytes, stp));
     JP_CUDA(launch_prof_classify_guide(j, ws, lg, st, pairs), "profile classify");
@@ -1380,7 +1382,7 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
   res->mode = select_mode_counts(p.n, p.raw_iters, p.war_iters, p.waw_iters, c.tau_high);
   res->n_tasks = 1;
   res->n_batches = 1;
-  return run_mode(L, j, res->mode, &p, c, ws, ws_bytes, res, st, gfuse && p.waw_iters == 0);
+  return run_mode(L, j, res->mode, &p, c, ws, ws_bytes, res, st, gfuse && p.waw_iters == 0, pairs);
 }
 
 
