@@ -177,6 +177,15 @@ def _cpu_model() -> str:
     return "unknown"
 
 
+def arm_config(world: int, n_per_rank: int) -> dict:
+    """The workload both arms report (the reference arm times the oracle on a
+    bounded sample of it; its cpu_baseline.sample says which)."""
+    return {"workload": "config2: DOALL streaming SAXPY fp32 Y=c0*X+Y, N=2^28, r=w=NULL",
+            "n_total": N2, "n_per_rank": n_per_rank, "partition": "task sharing, equal weights",
+            "l2": "inputs (3.2 GB) larger than L2 (126 MB); no flush needed",
+            "parallelism": f"iteration-range sharding x{world}"}
+
+
 def run_reference(args):
     """--impl reference: the oracle (the deliberately slow CPU program) on the
     host cores, each step a bounded 2^25-iteration sample of config 2."""
@@ -197,7 +206,7 @@ def run_reference(args):
                       "steps": args.steps, "warmup": args.warmup, "ms_per_step": t * 1e3,
                       "higher_is_better": True, "scaling": "strong", "vs_baseline": None, "dtype": "f32",
                       "data": "synthetic (synth.config2, seed 1002)",
-                      "config": {"workload": "config2: DOALL SAXPY fp32 N=2^28 (oracle on a 2^25-iteration sample)"},
+                      "config": arm_config(args.gpus, N2 // args.gpus),
                       "cpu_baseline": {"value": v, "unit": "iter/s", "cores": 1, "kind": "oracle",
                                        "sample": f"first {sample} iterations of config2 per step, jpo_run_seq, "
                                                  f"1 host thread of {os.cpu_count()}"},
@@ -691,10 +700,7 @@ def run_jp(args):
                "warmup": args.warmup, "ms_per_step": total_ms / args.steps, "higher_is_better": True,
                "scaling": "strong", "vs_baseline": None, "dtype": "f32",
                "data": "synthetic (synth.config2 counter-based generator, seed 1002), resident in HBM",
-               "config": {"workload": "config2: DOALL streaming SAXPY fp32 Y=c0*X+Y, N=2^28, r=w=NULL",
-                          "n_total": N2, "n_per_rank": s1 - s0, "partition": "task sharing, equal weights",
-                          "l2": "inputs (3.2 GB) larger than L2 (126 MB); no flush needed",
-                          "parallelism": f"iteration-range sharding x{world}"},
+               "config": arm_config(world, s1 - s0),
                "roofline": {"bound": "hbm", "kernel": ["k_doall_affine_vec<SAXPY,F32>",
                                                         "k_doall_affine_tma<SAXPY,F32>"][jp.jp_doall_kernel(-1)],
                             "achieved": achieved,
