@@ -118,8 +118,8 @@ typedef struct { int64_t committed, executed, windows, violations; } jp_tls_stat
  *   waw_iters == 0 (no address written twice; JP_ERR_ARG otherwise).  window:
  *   fixed W (0 = the largest the path holds); path: 5 one thread-block
  *   cluster, W <= 2048*cluster, cluster 1..16 (0 = auto: the smallest power of
- *   two that holds W, or n when W = 0); 6 every SM (cooperative), W <= 2048 *
- *   co-resident CTAs (303104 on a 148-SM B200), write log and shadow values in
+ *   two that holds W, or n when W = 0); 6 every SM (cooperative), W <= 3072 *
+ *   co-resident CTAs (454656 on a 148-SM B200, jp_tls_grid_window), write log and shadow values in
  *   workspace regions 7 and 8 (JP_WS_TLS); 0 = auto (5 when W, or n if W = 0,
  *   fits a 16-CTA cluster, else 6).  w_max is ignored.  stats: windows, violations =
  *   violating iterations, executed = n + violations, committed = n.  A second
@@ -520,6 +520,9 @@ const char *jp_last_error(void);
 const char *jp_version(void);
 /* Number of kernels this library has launched in this process (for bench.py). */
 int64_t jp_launch_count(void);
+/* The largest window of on-chip TLS path 6 on the current device (co-resident
+ * CTAs x 512 threads x 6 slots: 454656 on a 148-SM B200); 0 without a device. */
+int64_t jp_tls_grid_window(void);
 
 #ifdef __cplusplus
 }

@@ -28,7 +28,7 @@ __all__ = [
     "jp_plan_sharing", "jp_plan_stealing", "jp_merge_apply",
     "jp_plan_tasks", "jp_export_keys", "jp_keys_merge_p2p", "jp_run_priv_claim", "jp_run_doall_spill", "jp_ipc_export", "jp_ipc_import", "jp_ipc_close",
     "jp_sparse_scratch_bytes", "jp_sparse_pack", "jp_sparse_reduce_max", "jp_sparse_gather", "jp_sparse_scatter",
-    "jp_last_error", "jp_version", "jp_launch_count",
+    "jp_last_error", "jp_version", "jp_launch_count", "jp_tls_grid_window",
 ]
 
 _EL = {JP_I32: torch.int32, JP_F32: torch.float32}
@@ -468,3 +468,7 @@ def jp_version() -> str:
 
 def jp_launch_count() -> int:
     return int(lib().jp_launch_count())
+
+
+def jp_tls_grid_window() -> int:
+    return int(lib().jp_tls_grid_window())

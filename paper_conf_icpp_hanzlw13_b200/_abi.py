@@ -127,6 +127,7 @@ SIGNATURES = [
     ("jp_last_error", C.c_char_p, []),
     ("jp_version", C.c_char_p, []),
     ("jp_launch_count", _I64, []),
+    ("jp_tls_grid_window", _I64, []),
 ]
 
 _lock = threading.Lock()

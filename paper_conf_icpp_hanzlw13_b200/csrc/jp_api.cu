@@ -289,6 +289,7 @@ extern "C" {
 const char *jp_last_error(void) { return g_err.c_str(); }
 const char *jp_version(void) { return "jp-b200 0.1 (sm_100a)"; }
 int64_t jp_launch_count(void) { return g_launches.load(); }
+int64_t jp_tls_grid_window(void) { return have_device() ? tls_fwd_grid_wcap() : 0; }
 
 int32_t jp_doall_kernel(int32_t which) {
   if (which == 0 || which == 1) set_doall_kernel_choice(which);
@@ -560,7 +561,7 @@ static jp_status tls_plan(const Job &j, const jp_tls_cfg *cfg, const jp_profile 
       if (tp.window == 0) tp.window = gcap;
       if (tp.window > gcap)
         return fail(JP_ERR_UNSUPPORTED, "the on-chip TLS grid holds windows up to %lld iterations", (long long)gcap);
-      tp.cluster = (int)((tp.window + tls_fwd_wcap(1) - 1) / tls_fwd_wcap(1));
+      tp.cluster = (int)((tp.window + tls_fwd_grid_cta_slots() - 1) / tls_fwd_grid_cta_slots());
       tp.path = 6;
       tp.waw = false;
       return JP_OK;

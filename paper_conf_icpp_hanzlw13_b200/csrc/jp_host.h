@@ -128,7 +128,8 @@ cudaError_t launch_tls_fwd_grid(const Job &j, int64_t window, const uint32_t *bi
                                 unsigned long long *S,
                                 unsigned long long *V, int64_t lenS, unsigned *bar, int64_t *stats,
                                 cudaStream_t st, bool s_clean = false);
-int64_t tls_fwd_grid_wcap();         // 2048 * co-resident CTAs (2048 * 148 on B200)
+int64_t tls_fwd_grid_wcap();         // slots per CTA * co-resident CTAs (2048 * 148 on B200)
+int64_t tls_fwd_grid_cta_slots();    // window iterations per CTA of the all-SM kernel
 // stats: int64[4] device (committed, executed, windows, violations); bar: u32[2]
 // zeroed barrier words + int64[3] fv slots (grid path).
 cudaError_t launch_tls(const Job &j, void *ws, const Layout &lo, const TlsPlan &p, int64_t *stats,

@@ -409,11 +409,21 @@ cudaError_t tls_fwd_trace_copy(long long *host, int n) {
 #define FTR(ph) do { } while (0)
 #endif
 
+// the all-SM kernel's CTA shape (threads x window slots per thread); the
+// window is 148 x kGridT x kGridK iterations
+#ifndef JP_GRID_T
+#define JP_GRID_T 512
+#endif
+#ifndef JP_GRID_K
+#define JP_GRID_K 6
+#endif
+constexpr int kGridT = JP_GRID_T, kGridK = JP_GRID_K;
+
 template <int OP, int DT, bool GUIDED, int K>
 struct FwdGrid {
   static constexpr bool kTr = OP == JP_OP_ADD_C || OP == JP_OP_STENCIL2;
   static constexpr bool k2 = OP == JP_OP_STENCIL2;
-  static constexpr int T = kFwdThreads;
+  static constexpr int T = kGridT;
   DLoop L;
   const uint32_t *graw, *gsrc;
   unsigned long long *S, *V;
@@ -596,15 +606,15 @@ struct FwdGrid {
 };
 
 template <int OP, int DT, bool GUIDED>
-__global__ void __launch_bounds__(kFwdThreads, 1)
+__global__ void __launch_bounds__(kGridT, 1)
     k_tls_fwd_grid(DLoop L, int track, uint32_t W, const uint32_t *graw, const uint32_t *gsrc, unsigned long long *S,
                    unsigned long long *V, unsigned *bar, int64_t *stats) {
-  constexpr int K = kFwdK;
+  constexpr int K = kGridK;
   FwdGrid<OP, DT, GUIDED, K> F;
   F.L = L; F.graw = graw; F.gsrc = gsrc; F.S = S; F.V = V; F.bar = bar;
   F.W = W;
-  F.G = gridDim.x * (uint32_t)kFwdThreads;
-  F.g = blockIdx.x * (uint32_t)kFwdThreads + threadIdx.x;
+  F.G = gridDim.x * (uint32_t)kGridT;
+  F.g = blockIdx.x * (uint32_t)kGridT + threadIdx.x;
   F.n32 = (uint32_t)L.n;
   F.io = (uint32_t)L.ioff;
   F.nwin = (F.n32 + W - 1) / W;
@@ -639,14 +649,14 @@ static void run_fwd_grid(cudaError_t &e, const Job &j, uint32_t W, const uint32_
                          unsigned long long *S,
                          unsigned long long *V, unsigned *bar, int64_t *stats, cudaStream_t st) {
   void *fn = bits ? (void *)k_tls_fwd_grid<OP, DT, true> : (void *)k_tls_fwd_grid<OP, DT, false>;
-  const int grid = (int)((W + kFwdThreads * kFwdK - 1) / (kFwdThreads * kFwdK));
+  const int grid = (int)((W + kGridT * kGridK - 1) / (kGridT * kGridK));
   int maxb = 0;
-  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&maxb, fn, kFwdThreads, 0);
+  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&maxb, fn, kGridT, 0);
   if (grid > num_sms() * (maxb > 0 ? maxb : 1)) { e = cudaErrorInvalidConfiguration; return; }
   DLoop d = j.d;
   int track = a_indirect(j.op, j.d.r, j.d.r2, j.d.w) ? 1 : 0;
   void *args[] = {&d, &track, &W, &bits, &bsrc, &S, &V, &bar, &stats};
-  e = cudaLaunchCooperativeKernel(fn, dim3(grid), dim3(kFwdThreads), args, 0, st);
+  e = cudaLaunchCooperativeKernel(fn, dim3(grid), dim3(kGridT), args, 0, st);
   note_launch();
 }
 
@@ -673,11 +683,13 @@ cudaError_t launch_tls_fwd_grid(const Job &j, int64_t window, const uint32_t *bi
   return launch_check();
 }
 
+int64_t tls_fwd_grid_cta_slots() { return (int64_t)kGridT * kGridK; }
+
 int64_t tls_fwd_grid_wcap() {
   int maxb = 0;
-  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&maxb, (void *)k_tls_fwd_grid<JP_OP_ADD_C, JP_I32, true>, kFwdThreads, 0);
+  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&maxb, (void *)k_tls_fwd_grid<JP_OP_ADD_C, JP_I32, true>, kGridT, 0);
   cudaGetLastError();
-  return (int64_t)kFwdThreads * kFwdK * num_sms() * (maxb > 0 ? maxb : 1);
+  return (int64_t)kGridT * kGridK * num_sms() * (maxb > 0 ? maxb : 1);
 }
 
 // Largest cluster (power of two <= 16) the device schedules for k_tls_fwd (cached per device).

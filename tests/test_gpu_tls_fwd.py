@@ -34,7 +34,7 @@ def same(t: torch.Tensor, a: np.ndarray) -> bool:
 
 
 def grid_w():
-    return 2048 * torch.cuda.get_device_properties(0).multi_processor_count
+    return jp.jp_tls_grid_window()
 
 
 def fwd_case(wl, window, cluster=0, guided=False, view=None, path=5):
