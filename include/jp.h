@@ -392,8 +392,9 @@ jp_status jp_merge_apply(void *arr, int64_t len, const int64_t *keys, jp_stream_
  * jp_plan_tasks: chunk_counts (host [3 * ceil(n / chunk_iters)]: raw, war, waw
  * iteration counts of every chunk of the WHOLE loop L, e.g. the sum over the
  * ranks of jp_profile_classify's chunk counts) -> tasks = maximal runs of
- * chunks of one Fig. 2(b) mode (reading A19; at most 64, smaller runs merged
- * into the stronger mode), tasks (host [3 * 64]) = (start, end, mode) each,
+ * chunks of one Fig. 2(b) mode (reading A19; SEQ_RECOMMENDED kept as its own
+ * mode, run on the one-warp path 7; at most 64, smaller runs merged into the
+ * stronger mode, SEQ > TLS > PRIVATIZED > DOALL), tasks (host [3 * 64]) = (start, end, mode) each,
  * *n_tasks; conf (host [64]): bit t of conf[u] set iff tasks t and u touch a
  * common address and at least one writes it (reading B2), computed over L's
  * accesses on this device (workspace JP_WS_ALL of L).  chunk_iters >= 1024, a

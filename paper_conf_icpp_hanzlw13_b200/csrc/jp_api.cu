@@ -1046,12 +1046,13 @@ static std::vector<Task> chunk_tasks(const int64_t *hc, int64_t n, int64_t chunk
   const int64_t nck = (n + chunk - 1) / chunk;
   for (int64_t k = 0; k < nck; k++) {
     const int64_t s = k * chunk, e = std::min(n, s + chunk);
-    int m = select_mode_counts(e - s, hc[3 * k], hc[3 * k + 1], hc[3 * k + 2], tau);
-    if (m == JP_MODE_SEQ_RECOMMENDED) m = JP_MODE_TLS;
+    const int m = select_mode_counts(e - s, hc[3 * k], hc[3 * k + 1], hc[3 * k + 2], tau);
     if (!tasks.empty() && tasks.back().mode == m) tasks.back().e = e;
     else tasks.push_back({s, e, m});
   }
-  auto rank = [](int m) { return m == JP_MODE_TLS ? 2 : m == JP_MODE_PRIVATIZED ? 1 : 0; };
+  auto rank = [](int m) {
+    return m == JP_MODE_SEQ_RECOMMENDED ? 3 : m == JP_MODE_TLS ? 2 : m == JP_MODE_PRIVATIZED ? 1 : 0;
+  };
   while ((int)tasks.size() > kMaxTasks) {
     size_t best = 0;
     for (size_t q = 1; q + 1 < tasks.size(); q++)
@@ -1155,12 +1156,18 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
     for (int pass = 0; pass < 2; pass++) {
       for (int t = 0; t < nt; t++) {
         if (level[t] != lv) continue;
-        const bool tls = tasks[t].mode == JP_MODE_TLS;
+        const bool seq = tasks[t].mode == JP_MODE_SEQ_RECOMMENDED;
+        const bool tls = tasks[t].mode == JP_MODE_TLS || seq;
         if ((pass == 0) != tls) continue;
         cudaStream_t s2 = g_pool.get(sidx++);
         cudaStreamWaitEvent(s2, ev0, 0);
         Job sj = sub_job(j, tasks[t].s, tasks[t].e);
-        if (tls) {
+        if (seq && c.tls_path == 0 && c.tls_recovery == 0) {
+          // mode C task: one warp in program order (path 7) beside the partitioned tasks
+          JP_CUDA(launch_serial(sj, tstats + 4 * t, s2), "serial task");
+          res->tls_path = 7;
+          tls_tasks.push_back(t);
+        } else if (tls) {
           TlsPlan tp;
           jp_profile tprof{};
           tprof.n = sj.d.n;

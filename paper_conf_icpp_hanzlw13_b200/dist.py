@@ -386,7 +386,10 @@ def schedule_stealing(full, ws, group=None, chunk_iters: int = 65536, tau_high: 
                     waw = sum(ccl[3 * k + 2] for k in range(k0, k1))
                     tp = {"n": e2 - s, "raw_iters": raw, "war_iters": 0, "waw_iters": waw, "first_raw_iter": -1,
                           "d_raw": raw / max(e2 - s, 1), "d_war": 0.0, "d_waw": waw / max(e2 - s, 1)}
-                    st = jp.jp_run_tls(sub, prof=tp, ws=ws, recovery=int(waw == 0))
+                    if mode == _abi.JP_MODE_SEQ_RECOMMENDED:   # mode C: one warp, program order
+                        st = jp.jp_run_tls(sub, prof=tp, ws=ws, path=7)
+                    else:
+                        st = jp.jp_run_tls(sub, prof=tp, ws=ws, recovery=int(waw == 0))
                     for k in tls_stats:
                         tls_stats[k] += st[k]
                     jp.jp_export_keys(sub, ws)

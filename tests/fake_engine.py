@@ -249,7 +249,6 @@ def jp_plan_tasks(loop, chunk_counts, chunk_iters, ws, tau_high=0.25):
     for k in range(-(-n // chunk_iters)):
         s, e = k * chunk_iters, min(n, (k + 1) * chunk_iters)
         m = OS.select_mode(False, e - s, cc[3 * k], cc[3 * k + 1], cc[3 * k + 2], tau_high)
-        m = OS.TLS if m == OS.SEQ_RECOMMENDED else m
         if tasks and tasks[-1][2] == m:
             tasks[-1][1] = e
         else:

@@ -72,3 +72,18 @@ def region_workload(wl, b: int, e: int, name: str = None):
                           w=None if wl.w is None else wl.w[b:e].clone(),
                           s=None if wl.s is None else wl.s[b:e].clone(),
                           X=wl.X, T=None if wl.T is None else wl.T.clone(), c0=wl.c0, c1=wl.c1)
+
+
+def seq_mixed(n: int = 3 * 4096, seed: int = 9):
+    """ADD_C int32 over three equal regions with disjoint addresses: a permutation
+    (DOALL), a dependence chain r[i] = w[i-1] (d_raw = 100%: Fig. 2(b) mode C),
+    and a permutation again."""
+    assert n % 3 == 0
+    m = n // 3
+    g = np.random.default_rng(seed)
+    w = np.concatenate([g.permutation(m), m + np.arange(m), 2 * m + g.permutation(m)]).astype(np.int32)
+    r = w.copy()
+    r[m + 1:2 * m] = w[m:2 * m - 1]
+    A = g.integers(0, 1 << 20, size=n).astype(np.int32)
+    return synth.Workload("seq_mixed", O.OP_ADD_C, O.I32, n, torch.from_numpy(A), r=torch.from_numpy(r),
+                          w=torch.from_numpy(w), c0=7)

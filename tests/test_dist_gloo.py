@@ -103,7 +103,8 @@ def _jobs(world):
         share += [("share", c, "owner") for c in ("c1_5", "c4", "c5tail", "c5head")]
     else:
         share += [("share", "c5tail", "owner")]
-    steal = [("steal", "c5", "dense"), ("steal", "c5", "owner")] + ([("steal", "c1_5", "dense")] if world == 2 else [])
+    steal = [("steal", "c5", "dense"), ("steal", "c5", "owner")] + \
+        ([("steal", "c1_5", "dense"), ("steal", "seq", "dense")] if world == 2 else [])
     return share + steal
 
 
@@ -160,8 +161,9 @@ def _steal_case(rank, world, case, exchange, q):
         from paper_conf_icpp_hanzlw13_b200 import dist as jd
         import synth
         from helpers import to_oracle
+        from helpers import seq_mixed
         wl = {"c5": lambda: synth.config5(n=1 << 12, delta=64),
-              "c1_5": lambda: synth.config1(0.05, n=4096)}[case]()
+              "c1_5": lambda: synth.config1(0.05, n=4096), "seq": lambda: seq_mixed(3 * 1024)}[case]()
         ref = to_oracle(wl)
         _, A_exp, _ = O.run_seq(ref)
         full = jp.Loop.from_workload(wl)
@@ -176,11 +178,11 @@ def _steal_case(rank, world, case, exchange, q):
 
 
 @pytest.mark.parametrize("case,world,exchange", [("c5", 2, "dense"), ("c5", 3, "dense"), ("c5", 2, "owner"),
-                                                  ("c5", 3, "owner"), ("c1_5", 2, "dense")])
+                                                  ("c5", 3, "owner"), ("c1_5", 2, "dense"), ("seq", 2, "dense")])
 def test_stealing_scheme_matches_oracle(case, world, exchange):
     """Multi-rank task stealing (dist.schedule_stealing): partitioned profile with
     chunk counts, tasks + PDG, Alg. 1 plan, batches with C4 merges; every
     replica ends with the oracle's sequential result."""
     out = run_world(world, "steal", case, exchange)
     assert [o[1] for o in out] == [True] * world, out
-    assert sum(o[4] for o in out) == 4096
+    assert sum(o[4] for o in out) == (3 * 1024 if case == "seq" else 4096)

@@ -936,3 +936,17 @@ def test_schedule_host_pipelined_doall(op, dtype, n, chunk, monkeypatch):
     assert h["A"].numpy().tobytes() == A.tobytes()
     if T is not None:
         assert h["T"].numpy().tobytes() == T.tobytes()
+
+
+def test_schedule_stealing_mode_c_task():
+    """A chunk run above tau_high becomes a mode-C task of the stealing scheme and
+    runs on the one-warp program-order path beside the partitioned tasks."""
+    from helpers import seq_mixed
+    wl = seq_mixed(3 * 8192)
+    _, A, _ = O.run_seq(to_oracle(wl))
+    g = gpu(wl)
+    L = jp.Loop.from_workload(g)
+    res = jp.jp_schedule(L, jp.workspace(L), scheme=jp.JP_SCHED_STEALING, chunk_iters=2048)
+    torch.cuda.synchronize()
+    check_arrays(g, A, None)
+    assert res["task_mode_iters"][jp.JP_MODE_SEQ_RECOMMENDED] == 8192 and res["tls_path"] == 7, res
