@@ -8,6 +8,10 @@ with -fmad=false on both sides (BASELINE.json north_star; reading A12), so the
 bar is byte equality of every output array and exact integer statistics.
 """
 import itertools
+import os
+import shutil
+import subprocess
+import sys
 
 import numpy as np
 import pytest
@@ -950,3 +954,14 @@ def test_schedule_stealing_mode_c_task():
     torch.cuda.synchronize()
     check_arrays(g, A, None)
     assert res["task_mode_iters"][jp.JP_MODE_SEQ_RECOMMENDED] == 8192 and res["tls_path"] == 7, res
+
+
+@pytest.mark.skipif(shutil.which("compute-sanitizer") is None, reason="compute-sanitizer not on PATH")
+def test_memcheck_clean():
+    """compute-sanitizer memcheck over every kernel family at small N (scripts/sanitize.py):
+    no out-of-bounds or misaligned access, and every case still equals the oracle."""
+    root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+    out = subprocess.run(["compute-sanitizer", "--tool", "memcheck", "--print-limit", "5", sys.executable,
+                          os.path.join(root, "scripts", "sanitize.py")], capture_output=True, text=True, timeout=900)
+    assert "DONE fails=0" in out.stdout, out.stdout[-2000:] + out.stderr[-2000:]
+    assert "ERROR SUMMARY: 0 errors" in out.stdout + out.stderr, out.stdout[-2000:]
