@@ -98,6 +98,9 @@ _RESULTS = {}
 
 
 def _jobs(world):
+    if world == 4:
+        return [("share", "c4", "dense"), ("share", "c4", "owner"), ("share", "c5tail", "owner"),
+                ("share", "c3", "owner"), ("steal", "c5", "owner")]
     share = [("share", c, "dense") for c, _ in _CASES]
     if world == 3:
         share += [("share", c, "owner") for c in ("c1_5", "c4", "c5tail", "c5head")]
@@ -135,7 +138,9 @@ _CASES = [("c1_0", "DOALL"), ("c1_5", "TLS"), ("c4", "PRIVATIZED"), ("c3", "TLS"
 @pytest.mark.parametrize("world,case,mode,exchange",
                          [(w, c, m, "dense") for w in (2, 3) for c, m in _CASES] +
                          [(3, c, m, "owner") for c, m in _CASES if c in ("c1_5", "c4", "c5tail", "c5head")] +
-                         [(2, "c5tail", "PRIVATIZED", "owner")])
+                         [(2, "c5tail", "PRIVATIZED", "owner")] +
+                         [(4, "c4", "PRIVATIZED", "dense"), (4, "c4", "PRIVATIZED", "owner"),
+                          (4, "c5tail", "PRIVATIZED", "owner"), (4, "c3", "TLS", "owner")])
 def test_partitioned_schedule_matches_oracle(world, case, mode, exchange):
     out = run_world(world, "share", case, exchange)
     assert [o[1] for o in out] == [True] * world, out
@@ -178,7 +183,8 @@ def _steal_case(rank, world, case, exchange, q):
 
 
 @pytest.mark.parametrize("case,world,exchange", [("c5", 2, "dense"), ("c5", 3, "dense"), ("c5", 2, "owner"),
-                                                  ("c5", 3, "owner"), ("c1_5", 2, "dense"), ("seq", 2, "dense")])
+                                                  ("c5", 3, "owner"), ("c1_5", 2, "dense"), ("seq", 2, "dense"),
+                                                  ("c5", 4, "owner")])
 def test_stealing_scheme_matches_oracle(case, world, exchange):
     """Multi-rank task stealing (dist.schedule_stealing): partitioned profile with
     chunk counts, tasks + PDG, Alg. 1 plan, batches with C4 merges; every
