@@ -385,6 +385,22 @@ jp_status jp_schedule_workflow(const jp_loop *loops /* host [n] */, int32_t n, c
 /* Apply packed last-writer keys: arr[a] = keys[a] ? lo32(keys[a]) : arr[a]. */
 jp_status jp_merge_apply(void *arr, int64_t len, const int64_t *keys, jp_stream_t st);
 
+/* The scheduler's split plan entry (SURVEY §8(b) jp_plan; host only): from
+ * per-chunk profiles of the WHOLE loop (chunk_profiles host [n_chunks], chunk
+ * k = iterations [k*c, (k+1)*c), c = cfg->chunk_iters or 65536) to per-rank
+ * work.  Each chunk gets its Fig. 2(b) mode (cfg->tau_high); maximal runs of
+ * one mode are the tasks (reading A19).  cfg->scheme STEALING: the Alg. 1
+ * plan of jp_plan_stealing (TLS / mode-C tasks whole and pinned to rank 0,
+ * the others cut into chunks, dealt by task sharing, idle ranks stealing
+ * tails; speed_tls 1); SHARING: the boundary split of jp_plan_sharing, each
+ * rank's range cut at task boundaries.  plan_out (host [plan_cap][4]): rows
+ * (start, end, mode, owner); *n_out rows (JP_ERR_ARG with *n_out set when
+ * plan_cap is too small).  speed (host [world], nullable): per-rank weights.
+ * The inter-task PDG needs the loop's accesses: see jp_plan_tasks.          */
+jp_status jp_plan(const jp_loop *L, const jp_sched_cfg *cfg /* host */, const jp_profile *chunk_profiles /* host */,
+                  int64_t n_chunks, int32_t world, const double *speed /* host, nullable */,
+                  int64_t *plan_out /* host */, int64_t plan_cap, int64_t *n_out /* host */);
+
 /* ---- task stealing across ranks (SURVEY §8(e) "Mixed", Alg. 1) ----
  * The multi-rank stealing scheme (paper_conf_icpp_hanzlw13_b200/dist.py
  * schedule_stealing) needs, on every rank, the same task list and PDG that

@@ -26,7 +26,7 @@ __all__ = [
     "jp_profile_classify", "jp_profile_density", "jp_select_mode", "jp_run_doall", "jp_run_privatized",
     "jp_priv_stream", "jp_priv_finalize", "jp_doall_kernel", "jp_tls_guide", "tls_first_window", "jp_run_tls", "jp_schedule", "jp_stage_bytes", "jp_schedule_host",
     "jp_plan_sharing", "jp_plan_stealing", "jp_merge_apply",
-    "jp_plan_tasks", "jp_export_keys", "jp_keys_merge_p2p", "jp_run_priv_claim", "jp_run_doall_spill", "jp_ipc_export", "jp_ipc_import", "jp_ipc_close",
+    "jp_plan", "jp_plan_tasks", "jp_export_keys", "jp_keys_merge_p2p", "jp_run_priv_claim", "jp_run_doall_spill", "jp_ipc_export", "jp_ipc_import", "jp_ipc_close",
     "jp_sparse_scratch_bytes", "jp_sparse_pack", "jp_sparse_reduce_max", "jp_sparse_gather", "jp_sparse_scatter",
     "jp_last_error", "jp_version", "jp_launch_count", "jp_tls_grid_window",
 ]
@@ -351,6 +351,19 @@ def jp_merge_apply(arr: torch.Tensor, keys: torch.Tensor, stream=None):
 
 
 # ---- task stealing across ranks (jp.h) -------------------------------------
+def jp_plan(loop: Loop, chunk_profiles, world: int, speed=None, cfg=None, **kw):
+    """Host-only split plan (jp.h jp_plan): chunk_profiles = list of dicts (or
+    jp_profile) of the whole loop's chunks -> [(start, end, mode, owner)]."""
+    cfg = cfg if cfg is not None else sched_cfg(**kw)
+    arr = (_abi.jp_profile * max(len(chunk_profiles), 1))(*[_prof_struct(p) for p in chunk_profiles])
+    cap = 4 * (len(chunk_profiles) + world) + 8
+    out = (C.c_int64 * (4 * cap))()
+    n = C.c_int64()
+    sp = None if speed is None else (C.c_double * world)(*[float(x) for x in speed])
+    check(lib().jp_plan(loop.ref, C.byref(cfg), arr, len(chunk_profiles), int(world), sp, out, cap, C.byref(n)))
+    return [tuple(out[4 * k:4 * k + 4]) for k in range(n.value)]
+
+
 def jp_plan_tasks(loop: Loop, chunk_counts, chunk_iters: int, ws, tau_high: float = 0.25, stream=None):
     """chunk_counts: the whole loop's (raw, war, waw) per chunk (flat list / int64
     tensor).  Returns ([(start, end, mode)], conf list of 64 ints)."""

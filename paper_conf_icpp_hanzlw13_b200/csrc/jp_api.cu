@@ -1248,6 +1248,46 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
   return JP_OK;
 }
 
+jp_status jp_plan(const jp_loop *L, const jp_sched_cfg *cfg, const jp_profile *chunk_profiles, int64_t n_chunks,
+                  int32_t world, const double *speed, int64_t *plan_out, int64_t plan_cap, int64_t *n_out) {
+  JP_TRY(check_loop(L));
+  if (!cfg || !chunk_profiles || world <= 0 || !plan_out || !n_out)
+    return fail(JP_ERR_ARG, "bad plan arguments");
+  const int64_t chunk = cfg->chunk_iters > 0 ? cfg->chunk_iters : 65536;
+  if ((L->n + chunk - 1) / chunk != n_chunks)
+    return fail(JP_ERR_ARG, "%lld chunk profiles for %lld chunks of %lld iterations", (long long)n_chunks,
+                (long long)((L->n + chunk - 1) / chunk), (long long)chunk);
+  std::vector<int64_t> hc(3 * (size_t)std::max<int64_t>(n_chunks, 1));
+  for (int64_t k = 0; k < n_chunks; k++) {
+    hc[3 * k] = chunk_profiles[k].raw_iters;
+    hc[3 * k + 1] = chunk_profiles[k].war_iters;
+    hc[3 * k + 2] = chunk_profiles[k].waw_iters;
+  }
+  std::vector<Task> tk = chunk_tasks(hc.data(), L->n, chunk, cfg->tau_high > 0.0 ? cfg->tau_high : 0.25);
+  std::vector<int64_t> tasks;
+  for (const Task &t : tk) { tasks.push_back(t.s); tasks.push_back(t.e); tasks.push_back(t.mode); }
+  if (cfg->scheme == JP_SCHED_STEALING)
+    return jp_plan_stealing(tasks.data(), (int64_t)tk.size(), world, chunk, speed, 1.0, plan_out, plan_cap, n_out,
+                            nullptr);
+  // SHARING: the iteration space split by the boundary formula; each rank's range
+  // cut at task boundaries (rows keep one mode each)
+  std::vector<int64_t> rg(2 * (size_t)world);
+  JP_TRY(jp_plan_sharing(L->n, world, speed, rg.data()));
+  int64_t m = 0;
+  for (int k = 0; k < world; k++)
+    for (const Task &t : tk) {
+      const int64_t b = std::max(t.s, rg[2 * k]), e = std::min(t.e, rg[2 * k + 1]);
+      if (b >= e) continue;
+      if (m < plan_cap) {
+        plan_out[4 * m] = b; plan_out[4 * m + 1] = e; plan_out[4 * m + 2] = t.mode; plan_out[4 * m + 3] = k;
+      }
+      m++;
+    }
+  *n_out = m;
+  if (m > plan_cap) return fail(JP_ERR_ARG, "plan needs %lld rows", (long long)m);
+  return JP_OK;
+}
+
 jp_status jp_plan_tasks(const jp_loop *L, const int64_t *chunk_counts, int64_t chunk_iters, double tau_high,
                         void *ws, size_t ws_bytes, int64_t *tasks, int32_t *n_tasks, uint64_t *conf,
                         jp_stream_t st) {

@@ -8,6 +8,7 @@ import os
 import random
 import re
 
+import numpy as np
 import pytest
 import torch
 
@@ -226,3 +227,43 @@ def test_tls_first_window_matches_oracle(n, raw):
     bench path) equals the oracle's definition."""
     for w_max in (32, 4096, 65536):
         assert jp.tls_first_window(n, raw, w_max) == O.tls_next_window(n, raw, -1, w_max)
+
+
+@pytest.mark.parametrize("seed", range(12))
+def test_plan_matches_oracle_composition(seed):
+    """jp_plan (host split plan of SURVEY 8(b)): chunk modes by Fig. 2(b), maximal
+    same-mode runs, then the sharing split or the Alg. 1 plan -- against the
+    oracle's select_mode / sharing_ranges / stealing_plan composed in Python."""
+    import oracle.sched as OS
+    g = np.random.default_rng(seed)
+    chunk = 1024
+    nck = int(g.integers(1, 40))
+    n = nck * chunk - int(g.integers(0, chunk))
+    world = int(g.integers(1, 5))
+    profs, modes = [], []
+    for k in range(nck):
+        m = min(chunk, n - k * chunk)
+        kind = g.integers(0, 4)
+        raw = 0 if kind in (0, 1) else int(g.integers(1, m // 2 if kind == 2 else m))
+        war = int(g.integers(0, m)) if kind == 1 else 0
+        waw = int(g.integers(0, m)) if kind == 1 else 0
+        profs.append({"n": m, "raw_iters": raw, "war_iters": war, "waw_iters": waw, "first_raw_iter": -1,
+                      "d_raw": raw / m, "d_war": war / m, "d_waw": waw / m})
+        modes.append(OS.select_mode(False, m, raw, war, waw, 0.25))
+    tasks = []
+    for k, md in enumerate(modes):
+        s, e = k * chunk, min(n, (k + 1) * chunk)
+        if tasks and tasks[-1][2] == md:
+            tasks[-1][1] = e
+        else:
+            tasks.append([s, e, md])
+    A = torch.zeros(n, dtype=torch.int32)
+    L = jp.Loop(0, 0, n, A, r=torch.zeros(n, dtype=torch.int32), w=torch.zeros(n, dtype=torch.int32))
+    got = jp.jp_plan(L, profs, world, scheme=jp.JP_SCHED_STEALING, chunk_iters=chunk)
+    exp, _ = OS.stealing_plan([tuple(t) for t in tasks], world, chunk, None, 1.0)
+    assert [tuple(int(x) for x in r) for r in got] == [tuple(int(x) for x in r) for r in exp]
+    got = jp.jp_plan(L, profs, world, scheme=jp.JP_SCHED_SHARING, chunk_iters=chunk)
+    rg = OS.sharing_ranges(n, [1.0] * world)
+    exp = [(max(s, b), min(e, ee), md, k) for k, (b, ee) in enumerate(rg) for s, e, md in tasks
+           if max(s, b) < min(e, ee)]
+    assert [tuple(int(x) for x in r) for r in got] == exp
