@@ -496,8 +496,6 @@ struct FwdGrid {
     FTR(1);
     fwd_grid_sync(bar, gridDim.x * epoch);
     FTR(2);
-#pragma unroll
-    for (int k = 0; k < K; k++) dup += (uint32_t)(old[k] >> 32) == epoch;   // a second writer in this window
     // ---------------- this window's DC probes and the next window's forwarding
     // probes, all at once; the next window's gathers wait for the end of the
     // window so that probes and polls do not queue behind them ----------------
@@ -599,6 +597,10 @@ struct FwdGrid {
       }
     }
     if (more) gather(ws + W, nx, fwd);
+    // a second writer of an address in this window (checked last: the log
+    // atomics' return values must not hold up the probes issued after the barrier)
+#pragma unroll
+    for (int k = 0; k < K; k++) dup += (uint32_t)(old[k] >> 32) == epoch;
     FTR(7);
     if (win + 2 < nwin) load_idx(ws + 2 * W, c);
     FTR(8);
