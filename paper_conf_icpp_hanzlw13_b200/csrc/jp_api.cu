@@ -109,6 +109,7 @@ SchedLayout sched_layout(const jp_loop *L) {
   s.rmT = tI ? o : SIZE_MAX; if (tI) o = al256(o + 8 * (size_t)L->len_T);
   s.conf = o; o = al256(o + 8 * kMaxTasks);
   s.tstats = o; o = al256(o + 32 * kMaxTasks);
+  s.ranges = o; o = al256(o + 16 * kMaxTasks);
   s.total = o;
   return s;
 }
@@ -1080,6 +1081,22 @@ static jp_status task_conflicts(const Job &j, const jp_loop *L, void *ws, const 
     for (int64_t k = tasks[t].s / chunk; k * chunk < tasks[t].e; k++) ct[k] = t;
   int32_t *dct = reinterpret_cast<int32_t *>(sch + sl.chunk_task);
   JP_CUDA(cudaMemcpyAsync(dct, ct.data(), 4 * nck, cudaMemcpyHostToDevice, st), "task map H2D");
+  // cheap sufficient test first: tasks with disjoint address ranges in every array never conflict
+  if (!getenv("JP_TASK_MASKS_ALWAYS")) {
+    uint32_t *drg = reinterpret_cast<uint32_t *>(sch + sl.ranges);
+    JP_CUDA(launch_task_ranges(j, dct, chunk, drg, st), "task ranges");
+    std::vector<uint32_t> rg(4 * kMaxTasks);
+    JP_CUDA(cudaMemcpyAsync(rg.data(), drg, 16 * kMaxTasks, cudaMemcpyDeviceToHost, st), "ranges D2H");
+    JP_CUDA(cudaStreamSynchronize(st), "ranges sync");
+    auto ov = [&](int a, int t, int u) {   // array a: 0 A, 1 T
+      const uint32_t *mn = rg.data() + 2 * a * kMaxTasks, *mx = mn + kMaxTasks;
+      return mn[t] <= mx[t] && mn[u] <= mx[u] && !(mx[t] < mn[u] || mx[u] < mn[t]);
+    };
+    bool any = false;
+    for (int u = 0; u < nt && !any; u++)
+      for (int t = 0; t < u && !any; t++) any = ov(0, t, u) || ov(1, t, u);
+    if (!any) return JP_OK;   // conf stays all zero
+  }
   auto P = [&](size_t o) { return o == SIZE_MAX ? nullptr : reinterpret_cast<unsigned long long *>(sch + o); };
   unsigned long long *dconf = P(sl.conf);
   JP_CUDA(launch_task_conflicts(j, dct, chunk, nt, P(sl.wmA), P(sl.rmA), P(sl.wmT), P(sl.rmT), dconf, st),

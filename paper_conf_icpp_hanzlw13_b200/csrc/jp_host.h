@@ -27,7 +27,7 @@ constexpr int64_t kSchedMinChunk = 1024;
 constexpr int kMaxTasks = 64;
 // scheduler scratch sub-layout (inside R_SCHED)
 struct SchedLayout {
-  size_t counts, chunk_task, wmA, rmA, wmT, rmT, conf, tstats, total;
+  size_t counts, chunk_task, wmA, rmA, wmT, rmT, conf, tstats, ranges, total;
 };
 SchedLayout sched_layout(const jp_loop *L);
 
@@ -94,6 +94,8 @@ cudaError_t launch_sparse_rows(void *t0, void *t1, int elem, int64_t len, void *
 // STEALING scheduler helpers (jp_sched.cu): per-task write/read bitmasks of every
 // address, then the task x task conflict matrix conf[t] (bit u set: t and u
 // touch a common address and at least one of them writes it).
+// per-task address ranges rg [4][kMaxTasks] uint32 (minA, maxA, minT, maxT; empty: min > max)
+cudaError_t launch_task_ranges(const Job &j, const int32_t *chunk_task, int64_t chunk, uint32_t *rg, cudaStream_t st);
 cudaError_t launch_task_conflicts(const Job &j, const int32_t *chunk_task, int64_t chunk, int n_tasks,
                                   unsigned long long *wmA, unsigned long long *rmA,
                                   unsigned long long *wmT, unsigned long long *rmT,

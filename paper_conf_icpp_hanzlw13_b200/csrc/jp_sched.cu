@@ -100,6 +100,67 @@ __global__ void __launch_bounds__(256) k_task_conf(const unsigned long long *wm,
   if (threadIdx.x < kMaxTasks && sc[threadIdx.x]) atomicOr(&conf[threadIdx.x], sc[threadIdx.x]);
 }
 
+// Address range of every task per array (A, T): [min, max] over the elements
+// its iterations touch.  Tasks whose ranges are disjoint in every array cannot
+// touch a common address, so when no two ranges overlap the task PDG has no
+// edge and the per-address masks pass is skipped (one streaming pass over the
+// index arrays instead of two random atomics per access).  A warp's 32
+// iterations lie in one chunk (chunk % 32 == 0), hence in one task.
+template <int OP>
+__global__ void __launch_bounds__(256) k_task_ranges(DLoop L, const int32_t *ct, uint32_t chunk, uint32_t *rg) {
+  __shared__ uint32_t s[4][kMaxTasks];   // minA, maxA, minT, maxT
+  for (int t = threadIdx.x; t < kMaxTasks; t += blockDim.x) {
+    s[0][t] = s[2][t] = 0xFFFFFFFFu;
+    s[1][t] = s[3][t] = 0u;
+  }
+  __syncthreads();
+  const int lane = threadIdx.x & 31;
+  const int64_t nw = (int64_t)gridDim.x * (blockDim.x >> 5);
+  for (int64_t base = ((int64_t)blockIdx.x * (blockDim.x >> 5) + (threadIdx.x >> 5)) * 32; base < L.n; base += nw * 32) {
+    const int64_t i = base + lane;
+    uint32_t amin = 0xFFFFFFFFu, amax = 0u, tmin = 0xFFFFFFFFu, tmax = 0u;
+    if (i < L.n) {
+      auto acc = [&](int64_t a) { amin = min(amin, (uint32_t)a); amax = max(amax, (uint32_t)a); };
+      acc(ixl(L, L.w, i));
+      if constexpr (OP == JP_OP_ADD_C || OP == JP_OP_STENCIL2) acc(ixl(L, L.r, i));
+      if constexpr (OP == JP_OP_STENCIL2) acc(ixl(L, L.r2, i));
+      if constexpr (OP == JP_OP_PRIV_TMP) { tmin = tmax = (uint32_t)ixl(L, L.s, i); }
+    }
+    amin = __reduce_min_sync(0xffffffffu, amin);
+    amax = __reduce_max_sync(0xffffffffu, amax);
+    tmin = __reduce_min_sync(0xffffffffu, tmin);
+    tmax = __reduce_max_sync(0xffffffffu, tmax);
+    if (lane == 0) {
+      const int t = ct[base / chunk];
+      atomicMin(&s[0][t], amin); atomicMax(&s[1][t], amax);
+      atomicMin(&s[2][t], tmin); atomicMax(&s[3][t], tmax);
+    }
+  }
+  __syncthreads();
+  for (int t = threadIdx.x; t < kMaxTasks; t += blockDim.x) {
+    if (s[0][t] != 0xFFFFFFFFu) { atomicMin(&rg[t], s[0][t]); atomicMax(&rg[kMaxTasks + t], s[1][t]); }
+    if (s[2][t] != 0xFFFFFFFFu) { atomicMin(&rg[2 * kMaxTasks + t], s[2][t]); atomicMax(&rg[3 * kMaxTasks + t], s[3][t]); }
+  }
+}
+
+template <int OP, int DT>
+static void run_ranges(const DLoop &d, const int32_t *ct, int64_t chunk, uint32_t *rg, cudaStream_t st) {
+  (void)DT;
+  int64_t need = (d.n + 255) / 256, cap = (int64_t)num_sms() * 4;
+  k_task_ranges<OP><<<(int)(need < cap ? (need < 1 ? 1 : need) : cap), 256, 0, st>>>(d, ct, (uint32_t)chunk, rg);
+  note_launch();
+}
+
+cudaError_t launch_task_ranges(const Job &j, const int32_t *chunk_task, int64_t chunk, uint32_t *rg, cudaStream_t st) {
+  cudaMemsetAsync(rg, 0xFF, 4 * kMaxTasks, st);
+  cudaMemsetAsync(rg + kMaxTasks, 0, 4 * kMaxTasks, st);
+  cudaMemsetAsync(rg + 2 * kMaxTasks, 0xFF, 4 * kMaxTasks, st);
+  cudaMemsetAsync(rg + 3 * kMaxTasks, 0, 4 * kMaxTasks, st);
+  if (j.d.n == 0) return launch_check();
+  JP_DISPATCH(j.op, j.dt, run_ranges, j.d, chunk_task, chunk, rg, st);
+  return launch_check();
+}
+
 template <int OP, int DT>
 static void run_masks(const DLoop &d, const int32_t *ct, int64_t chunk, unsigned long long *wmA,
                       unsigned long long *rmA, unsigned long long *wmT, unsigned long long *rmT, bool b8,

@@ -886,13 +886,16 @@ def test_schedule_mode_c_runs_serial(case):
         assert res["task_mode_iters"][jp.JP_MODE_SEQ_RECOMMENDED] == n
 
 
+@pytest.mark.parametrize("masks_always", ["0", "1"])
 @pytest.mark.parametrize("seed", range(6))
-def test_plan_tasks_matches_definition(seed):
+def test_plan_tasks_matches_definition(seed, masks_always, monkeypatch):
     """jp_plan_tasks (tasks = maximal same-mode chunk runs, PDG from per-address
     task masks) against its plain definition (tests/fake_engine.py: Fig. 2(b)
     per chunk via oracle/sched.select_mode, address sets per task, pairwise
     intersection) on loops mixing DOALL / privatized / TLS regions."""
     import fake_engine as fe
+    if masks_always == "1":   # skip the address-range prefilter: the masks pass decides every pair
+        monkeypatch.setenv("JP_TASK_MASKS_ALWAYS", "1")
     g = np.random.default_rng(seed)
     n, chunk = 8192, 1024
     if seed % 2:
