@@ -1121,8 +1121,10 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
   const bool gfuse = lo.bytes[R_GUIDE] && c.tls_recovery != 1 && j.op != JP_OP_PRIV_TMP &&
                      a_indirect(j.op, j.d.r, j.d.r2, j.d.w);
   uint32_t *gbits = gfuse ? at<uint32_t>(ws, lo, R_GUIDE) : nullptr;
-  JP_CUDA(launch_prof_stamp(j, ws, lo, st), "profile stamp");
-  JP_CUDA(launch_prof_classify(j, ws, lo, gbits, chunk, cc, st, gbits ? gbits + (L->n + 31) / 32 : nullptr),
+  // large A tables: stamped as {minW, minR} pairs in region 7 (free until the TLS tasks run)
+  const bool pairs = stamp_pairs_ok(j, ws, lo);
+  JP_CUDA(launch_prof_stamp(j, ws, lo, st, pairs), "profile stamp");
+  JP_CUDA(launch_prof_classify(j, ws, lo, gbits, chunk, cc, st, gbits ? gbits + (L->n + 31) / 32 : nullptr, pairs),
           "profile classify");
   std::vector<int64_t> hc(3 * nck), h(8);
   JP_CUDA(cudaMemcpyAsync(hc.data(), cc, 24 * nck, cudaMemcpyDeviceToHost, st), "chunk D2H");

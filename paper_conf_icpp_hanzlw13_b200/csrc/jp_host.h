@@ -52,7 +52,8 @@ cudaError_t launch_prof_stamp(const Job &j, void *ws, const Layout &lo, cudaStre
 bool stamp_pairs_ok(const Job &j, void *ws, const Layout &lo);
 // src_bits (nullable): also the TLS guide's RAW-source words (raw_bits then holds its raw words)
 cudaError_t launch_prof_classify(const Job &j, void *ws, const Layout &lo, uint32_t *raw_bits,
-                                 int64_t chunk, int64_t *chunk_counts, cudaStream_t st, uint32_t *src_bits = nullptr);
+                                 int64_t chunk, int64_t *chunk_counts, cudaStream_t st, uint32_t *src_bits = nullptr,
+                                 bool stamped_pairs = false);
 // counts + the TLS guide bitmaps (region 13, valid when the loop writes no address twice) in one pass
 cudaError_t launch_prof_classify_guide(const Job &j, void *ws, const Layout &lo, cudaStream_t st,
                                        bool stamped_pairs = false);

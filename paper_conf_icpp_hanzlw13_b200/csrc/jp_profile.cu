@@ -319,8 +319,8 @@ static int idx_vec(const DLoop &d) {
 }
 
 // (bounds-guarded: classify may run before the host has seen the bad-index count)
-__device__ __forceinline__ bool earlier(const int32_t *tab, int64_t a, int64_t len, int32_t e) {
-  return tab && (uint64_t)a < (uint64_t)len && tab[a] > e;
+__device__ __forceinline__ bool earlier(const int32_t *tab, int64_t a, int64_t len, int32_t e, int stride = 1) {
+  return tab && (uint64_t)a < (uint64_t)len && tab[a * stride] > e;
 }
 
 // src_bits (nullable, zeroed by the caller): the RAW-source words of the TLS
@@ -362,28 +362,28 @@ __global__ void __launch_bounds__(256) k_prof_classify(DLoop L, Tabs t, uint32_t
         const int32_t e = enc_gid(L.base + i);
         auto src = [&](int64_t a) {   // mark the first writer of a raw read's address
           if (src_bits) {
-            const int64_t jw = (int64_t)(0x7FFFFFFF - t.wA[a]) - L.base;
+            const int64_t jw = (int64_t)(0x7FFFFFFF - t.wA[(int64_t)a * t.as]) - L.base;
             atomicOr(&src_bits[jw >> 5], 1u << (jw & 31));
           }
         };
         if constexpr (OP == JP_OP_ADD_C) {
-          war[u] = earlier(t.rA, ia[u], L.lenA, e);
-          waw[u] = earlier(t.wA, ia[u], L.lenA, e);
-          raw[u] = ib[u] == ia[u] ? waw[u] : earlier(t.wA, ib[u], L.lenA, e);   // r == w: one lookup
+          war[u] = earlier(t.rA, ia[u], L.lenA, e, t.as);
+          waw[u] = earlier(t.wA, ia[u], L.lenA, e, t.as);
+          raw[u] = ib[u] == ia[u] ? waw[u] : earlier(t.wA, ib[u], L.lenA, e, t.as);   // r == w: one lookup
           if (raw[u]) src(ib[u]);
         } else if constexpr (OP == JP_OP_SAXPY) {
-          raw[u] = earlier(t.wA, ia[u], L.lenA, e);
-          war[u] = earlier(t.rA, ia[u], L.lenA, e);
+          raw[u] = earlier(t.wA, ia[u], L.lenA, e, t.as);
+          war[u] = earlier(t.rA, ia[u], L.lenA, e, t.as);
           waw[u] = raw[u];   // the same address is the exposed read and the write
           if (raw[u]) src(ia[u]);
         } else if constexpr (OP == JP_OP_PRIV_TMP) {
           war[u] = earlier(rT, ia[u], L.lenT, e);
-          waw[u] = earlier(t.wT, ia[u], L.lenT, e) || earlier(t.wA, ib[u], L.lenA, e);
+          waw[u] = earlier(t.wT, ia[u], L.lenT, e) || earlier(t.wA, ib[u], L.lenA, e, t.as);
         } else {
-          war[u] = earlier(t.rA, ia[u], L.lenA, e);
-          waw[u] = earlier(t.wA, ia[u], L.lenA, e);
-          const bool r0 = ib[u] == ia[u] ? waw[u] : earlier(t.wA, ib[u], L.lenA, e);
-          const bool r1 = ic[u] == ia[u] ? waw[u] : ic[u] == ib[u] ? r0 : earlier(t.wA, ic[u], L.lenA, e);
+          war[u] = earlier(t.rA, ia[u], L.lenA, e, t.as);
+          waw[u] = earlier(t.wA, ia[u], L.lenA, e, t.as);
+          const bool r0 = ib[u] == ia[u] ? waw[u] : earlier(t.wA, ib[u], L.lenA, e, t.as);
+          const bool r1 = ic[u] == ia[u] ? waw[u] : ic[u] == ib[u] ? r0 : earlier(t.wA, ic[u], L.lenA, e, t.as);
           raw[u] = r0 || r1;
           if (r0) src(ib[u]);
           if (r1) src(ic[u]);
@@ -601,13 +601,18 @@ static void run_classify(const DLoop &d, Tabs t, uint32_t *bits, int64_t chunk, 
 }
 
 cudaError_t launch_prof_classify(const Job &j, void *ws, const Layout &lo, uint32_t *raw_bits, int64_t chunk,
-                                 int64_t *chunk_counts, cudaStream_t st, uint32_t *src_bits) {
+                                 int64_t *chunk_counts, cudaStream_t st, uint32_t *src_bits, bool stamped_pairs) {
   int64_t *hdr = at<int64_t>(ws, lo, R_HEADER);
   cudaMemsetAsync(&hdr[H_RAW], 0, 3 * sizeof(int64_t), st);
   cudaMemsetAsync(&hdr[H_FIRST_RAW], 0xFF, sizeof(int64_t), st);
   if (chunk_counts) cudaMemsetAsync(chunk_counts, 0, sizeof(int64_t) * 3 * ((j.d.n + chunk - 1) / chunk), st);
   if (j.d.n == 0) return launch_check();
   Tabs t = tabs_of(j.d, ws, lo);
+  if (stamped_pairs) {   // the stamp pass wrote {minW, minR} pairs into region 7
+    t.wA = at<int32_t>(ws, lo, R_TLS_S_A);
+    t.rA = t.wA + 1;
+    t.as = 2;
+  }
   if (src_bits) cudaMemsetAsync(src_bits, 0, 4 * (size_t)((j.d.n + 31) / 32), st);
   JP_DISPATCH(j.op, j.dt, run_classify, j.d, t, raw_bits, chunk, chunk_counts, hdr, src_bits, st);
   return launch_check();
