@@ -1067,10 +1067,13 @@ static std::vector<Task> chunk_tasks(const int64_t *hc, int64_t n, int64_t chunk
 }
 
 // conf[u] bit t: tasks t and u touch a common address, at least one writing it (reading B2); syncs
+// ranges_out (nullable): the per-task address ranges of the prefilter
+// ([4][kMaxTasks]: minA, maxA, minT, maxT) when it ran, else left empty
 static jp_status task_conflicts(const Job &j, const jp_loop *L, void *ws, const Layout &lo,
                                 const std::vector<Task> &tasks, int64_t chunk, std::vector<unsigned long long> &conf,
-                                cudaStream_t st) {
+                                cudaStream_t st, std::vector<uint32_t> *ranges_out = nullptr) {
   const int nt = (int)tasks.size();
+  if (ranges_out) ranges_out->clear();
   conf.assign(kMaxTasks, 0);
   if (nt <= 1) return JP_OK;
   SchedLayout sl = sched_layout(L);
@@ -1088,6 +1091,7 @@ static jp_status task_conflicts(const Job &j, const jp_loop *L, void *ws, const 
     std::vector<uint32_t> rg(4 * kMaxTasks);
     JP_CUDA(cudaMemcpyAsync(rg.data(), drg, 16 * kMaxTasks, cudaMemcpyDeviceToHost, st), "ranges D2H");
     JP_CUDA(cudaStreamSynchronize(st), "ranges sync");
+    if (ranges_out) *ranges_out = rg;
     auto ov = [&](int a, int t, int u) {   // array a: 0 A, 1 T
       const uint32_t *mn = rg.data() + 2 * a * kMaxTasks, *mx = mn + kMaxTasks;
       return mn[t] <= mx[t] && mn[u] <= mx[u] && !(mx[t] < mn[u] || mx[u] < mn[t]);
@@ -1140,7 +1144,8 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
   res->mode = nt ? tasks[0].mode : JP_MODE_DOALL;
   // 3. inter-task conflicts (PDG) and topological batches
   std::vector<unsigned long long> conf(kMaxTasks, 0);
-  JP_TRY(task_conflicts(j, L, ws, lo, tasks, chunk, conf, st));
+  std::vector<uint32_t> trg;
+  JP_TRY(task_conflicts(j, L, ws, lo, tasks, chunk, conf, st, &trg));
   std::vector<int> level(nt, 0);
   int nlev = nt ? 1 : 0;
   for (int u = 0; u < nt; u++) {
@@ -1164,9 +1169,29 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
   for (int lv = 0; lv < nlev; lv++) {
     bool any_priv = false;
     for (int t = 0; t < nt; t++) any_priv |= level[t] == lv && tasks[t].mode == JP_MODE_PRIVATIZED;
+    // the element ranges this batch's privatized tasks can write (their keys):
+    // the whole arrays unless the range prefilter ran
+    int64_t kA0 = 0, kA1 = L->len_A, kT0 = 0, kT1 = L->len_T;
+    if (any_priv && !trg.empty()) {
+      kA0 = kT0 = INT64_MAX;
+      kA1 = kT1 = 0;
+      for (int t = 0; t < nt; t++) {
+        if (level[t] != lv || tasks[t].mode != JP_MODE_PRIVATIZED) continue;
+        const uint32_t *r = trg.data();
+        if (r[t] <= r[kMaxTasks + t]) { kA0 = std::min<int64_t>(kA0, r[t]); kA1 = std::max<int64_t>(kA1, (int64_t)r[kMaxTasks + t] + 1); }
+        if (r[2 * kMaxTasks + t] <= r[3 * kMaxTasks + t]) {
+          kT0 = std::min<int64_t>(kT0, r[2 * kMaxTasks + t]);
+          kT1 = std::max<int64_t>(kT1, (int64_t)r[3 * kMaxTasks + t] + 1);
+        }
+      }
+      if (kA0 >= kA1) kA0 = kA1 = 0;
+      if (kT0 >= kT1) kT0 = kT1 = 0;
+    }
+    auto *keysA = at<unsigned long long>(ws, lo, R_KEYS_A);
+    auto *keysT = at<unsigned long long>(ws, lo, R_KEYS_T);
     if (any_priv) {
-      if (lo.bytes[R_KEYS_A]) cudaMemsetAsync(at<char>(ws, lo, R_KEYS_A), 0, lo.bytes[R_KEYS_A], st);
-      if (lo.bytes[R_KEYS_T]) cudaMemsetAsync(at<char>(ws, lo, R_KEYS_T), 0, lo.bytes[R_KEYS_T], st);
+      if (keysA && kA1 > kA0) cudaMemsetAsync(keysA + kA0, 0, 8 * (size_t)(kA1 - kA0), st);
+      if (keysT && kT1 > kT0) cudaMemsetAsync(keysT + kT0, 0, 8 * (size_t)(kT1 - kT0), st);
     }
     cudaEventRecord(ev0, st);
     int sidx = 0;
@@ -1251,7 +1276,14 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
       res->tls_guided = gb ? 1 : 0;
       tls_tasks.push_back(t);
     }
-    if (any_priv) JP_CUDA(launch_priv_finalize(j, ws, lo, st), "priv finalize");
+    if (any_priv) {   // apply the keys over the written ranges only
+      if (keysA && kA1 > kA0)
+        JP_CUDA(launch_merge_apply(static_cast<uint32_t *>(L->A) + kA0, kA1 - kA0,
+                                   reinterpret_cast<const int64_t *>(keysA + kA0), st), "priv finalize");
+      if (keysT && kT1 > kT0 && j.op == JP_OP_PRIV_TMP)
+        JP_CUDA(launch_merge_apply(static_cast<uint32_t *>(L->T) + kT0, kT1 - kT0,
+                                   reinterpret_cast<const int64_t *>(keysT + kT0), st), "priv finalize");
+    }
   }
   // stats of the TLS tasks
   memset(&res->tls, 0, sizeof res->tls);

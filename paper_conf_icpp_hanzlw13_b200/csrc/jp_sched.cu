@@ -115,27 +115,59 @@ __global__ void __launch_bounds__(256) k_task_ranges(DLoop L, const int32_t *ct,
   }
   __syncthreads();
   const int lane = threadIdx.x & 31;
-  const int64_t nw = (int64_t)gridDim.x * (blockDim.x >> 5);
-  for (int64_t base = ((int64_t)blockIdx.x * (blockDim.x >> 5) + (threadIdx.x >> 5)) * 32; base < L.n; base += nw * 32) {
-    const int64_t i = base + lane;
-    uint32_t amin = 0xFFFFFFFFu, amax = 0u, tmin = 0xFFFFFFFFu, tmax = 0u;
-    if (i < L.n) {
-      auto acc = [&](int64_t a) { amin = min(amin, (uint32_t)a); amax = max(amax, (uint32_t)a); };
-      acc(ixl(L, L.w, i));
-      if constexpr (OP == JP_OP_ADD_C || OP == JP_OP_STENCIL2) acc(ixl(L, L.r, i));
-      if constexpr (OP == JP_OP_STENCIL2) acc(ixl(L, L.r2, i));
-      if constexpr (OP == JP_OP_PRIV_TMP) { tmin = tmax = (uint32_t)ixl(L, L.s, i); }
+  // each warp streams a contiguous run of 32-iteration tiles, keeping its
+  // min / max in registers while the task stays the same (one warp reduction
+  // per task change instead of one per tile)
+  const int64_t tiles = (L.n + 31) / 32, nw = (int64_t)gridDim.x * (blockDim.x >> 5);
+  const int64_t wg = (int64_t)blockIdx.x * (blockDim.x >> 5) + (threadIdx.x >> 5);
+  const int64_t t0 = tiles * wg / nw, t1 = tiles * (wg + 1) / nw;
+  uint32_t amin = 0xFFFFFFFFu, amax = 0u, tmin = 0xFFFFFFFFu, tmax = 0u;
+  int cur = t0 < t1 ? ct[(t0 * 32) / chunk] : -1;
+  auto flush = [&]() {
+    const uint32_t a0 = __reduce_min_sync(0xffffffffu, amin), a1 = __reduce_max_sync(0xffffffffu, amax);
+    const uint32_t b0 = __reduce_min_sync(0xffffffffu, tmin), b1 = __reduce_max_sync(0xffffffffu, tmax);
+    if (lane == 0 && cur >= 0) {
+      atomicMin(&s[0][cur], a0); atomicMax(&s[1][cur], a1);
+      atomicMin(&s[2][cur], b0); atomicMax(&s[3][cur], b1);
     }
-    amin = __reduce_min_sync(0xffffffffu, amin);
-    amax = __reduce_max_sync(0xffffffffu, amax);
-    tmin = __reduce_min_sync(0xffffffffu, tmin);
-    tmax = __reduce_max_sync(0xffffffffu, tmax);
-    if (lane == 0) {
-      const int t = ct[base / chunk];
-      atomicMin(&s[0][t], amin); atomicMax(&s[1][t], amax);
-      atomicMin(&s[2][t], tmin); atomicMax(&s[3][t], tmax);
+    amin = tmin = 0xFFFFFFFFu;
+    amax = tmax = 0u;
+  };
+  constexpr int U = 8;   // tiles whose loads are in flight together
+  auto tile_acc = [&](int64_t tile0, int nt) {
+    uint32_t w[U], r[U], x[U];
+#pragma unroll
+    for (int u = 0; u < U; u++) {   // all loads first
+      const int64_t i = (tile0 + u) * 32 + lane;
+      w[u] = r[u] = x[u] = 0;
+      if (u < nt && i < L.n) {
+        w[u] = (uint32_t)ixl(L, L.w, i);
+        if constexpr (OP == JP_OP_ADD_C || OP == JP_OP_STENCIL2) r[u] = (uint32_t)ixl(L, L.r, i);
+        if constexpr (OP == JP_OP_STENCIL2 || OP == JP_OP_PRIV_TMP)
+          x[u] = (uint32_t)ixl(L, OP == JP_OP_STENCIL2 ? L.r2 : L.s, i);
+      }
     }
+#pragma unroll
+    for (int u = 0; u < U; u++) {
+      const int64_t i = (tile0 + u) * 32 + lane;
+      if (u < nt && i < L.n) {
+        amin = min(amin, w[u]); amax = max(amax, w[u]);
+        if constexpr (OP == JP_OP_ADD_C || OP == JP_OP_STENCIL2) { amin = min(amin, r[u]); amax = max(amax, r[u]); }
+        if constexpr (OP == JP_OP_STENCIL2) { amin = min(amin, x[u]); amax = max(amax, x[u]); }
+        if constexpr (OP == JP_OP_PRIV_TMP) { tmin = min(tmin, x[u]); tmax = max(tmax, x[u]); }
+      }
+    }
+  };
+  for (int64_t tile = t0; tile < t1;) {
+    const int task = ct[(tile * 32) / chunk];   // warp-uniform (chunk % 32 == 0)
+    if (task != cur) { flush(); cur = task; }
+    // U tiles at once when they all lie in this task (tasks are runs of chunks)
+    int nt = 1;
+    if (tile + U <= t1 && ct[((tile + U - 1) * 32) / chunk] == task) nt = U;
+    tile_acc(tile, nt);
+    tile += nt;
   }
+  flush();
   __syncthreads();
   for (int t = threadIdx.x; t < kMaxTasks; t += blockDim.x) {
     if (s[0][t] != 0xFFFFFFFFu) { atomicMin(&rg[t], s[0][t]); atomicMax(&rg[kMaxTasks + t], s[1][t]); }
@@ -146,7 +178,7 @@ __global__ void __launch_bounds__(256) k_task_ranges(DLoop L, const int32_t *ct,
 template <int OP, int DT>
 static void run_ranges(const DLoop &d, const int32_t *ct, int64_t chunk, uint32_t *rg, cudaStream_t st) {
   (void)DT;
-  int64_t need = (d.n + 255) / 256, cap = (int64_t)num_sms() * 4;
+  int64_t need = (d.n + 255) / 256, cap = (int64_t)num_sms() * 8;
   k_task_ranges<OP><<<(int)(need < cap ? (need < 1 ? 1 : need) : cap), 256, 0, st>>>(d, ct, (uint32_t)chunk, rg);
   note_launch();
 }
