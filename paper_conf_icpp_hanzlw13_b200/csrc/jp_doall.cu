@@ -161,6 +161,77 @@ __global__ void __launch_bounds__(256) k_doall_generic(DLoop L) {
   }
 }
 
+// k_doall_quad: the indirect DOALL body with more random accesses in flight --
+// each thread takes two quads of 4 consecutive iterations per trip (16-byte
+// index loads when aligned), issues all 8 iterations' gathers, then computes
+// and scatters.  The loop carries no dependence (d_raw = d_war = d_waw = 0), so
+// reading A in place and storing in any order is the sequential result.
+__device__ __forceinline__ int4 q_idx(const DLoop &L, const int32_t *p, int64_t i, bool vec) {
+  if (!p) {
+    const int32_t b = (int32_t)(L.ioff + i);
+    return make_int4(b, b + 1, b + 2, b + 3);
+  }
+  if (vec && i + 4 <= L.n) return __ldcs(reinterpret_cast<const int4 *>(p + i));
+  int4 r;
+  r.x = p[i];
+  r.y = i + 1 < L.n ? p[i + 1] : 0;
+  r.z = i + 2 < L.n ? p[i + 2] : 0;
+  r.w = i + 3 < L.n ? p[i + 3] : 0;
+  return r;
+}
+__device__ __forceinline__ int q_get(const int4 &v, int k) { return k == 0 ? v.x : k == 1 ? v.y : k == 2 ? v.z : v.w; }
+
+template <int OP, int DT>
+__global__ void __launch_bounds__(256) k_doall_quad(DLoop L, int vec) {
+  constexpr int Q = 2;   // quads per thread per trip
+  const int64_t nq = (L.n + 3) >> 2, B = blockDim.x;
+  for (int64_t q0 = (int64_t)blockIdx.x * B * Q + threadIdx.x; q0 < nq; q0 += (int64_t)gridDim.x * B * Q) {
+    int4 ra[Q], wa[Q], xa[Q];
+    uint32_t g0[Q][4], g1[Q][4];
+#pragma unroll
+    for (int u = 0; u < Q; u++) {
+      const int64_t q = q0 + u * B;
+      if (q >= nq) continue;
+      const int64_t i = q << 2;
+      ra[u] = q_idx(L, L.r, i, vec);
+      wa[u] = q_idx(L, L.w, i, vec);
+      if constexpr (OP == JP_OP_STENCIL2) xa[u] = q_idx(L, L.r2, i, vec);
+      if constexpr (OP == JP_OP_PRIV_TMP) xa[u] = q_idx(L, L.s, i, vec);
+    }
+#pragma unroll
+    for (int u = 0; u < Q; u++) {   // every gather of the trip issued before any use
+      const int64_t q = q0 + u * B;
+      if (q >= nq) continue;
+      const int kn = L.n - (q << 2) < 4 ? (int)(L.n - (q << 2)) : 4;
+#pragma unroll
+      for (int k = 0; k < 4; k++) {
+        if (k >= kn) break;
+        if constexpr (OP == JP_OP_ADD_C) g0[u][k] = L.A[q_get(ra[u], k)];
+        else if constexpr (OP == JP_OP_SAXPY) { g0[u][k] = L.X[q_get(ra[u], k)]; g1[u][k] = L.A[q_get(wa[u], k)]; }
+        else if constexpr (OP == JP_OP_PRIV_TMP) g0[u][k] = L.X[q_get(ra[u], k)];
+        else { g0[u][k] = L.A[q_get(ra[u], k)]; g1[u][k] = L.A[q_get(xa[u], k)]; }
+      }
+    }
+#pragma unroll
+    for (int u = 0; u < Q; u++) {
+      const int64_t q = q0 + u * B;
+      if (q >= nq) continue;
+      const int kn = L.n - (q << 2) < 4 ? (int)(L.n - (q << 2)) : 4;
+#pragma unroll
+      for (int k = 0; k < 4; k++) {
+        if (k >= kn) break;
+        if constexpr (OP == JP_OP_ADD_C) L.A[q_get(wa[u], k)] = op_add<DT>(g0[u][k], L.c0);
+        else if constexpr (OP == JP_OP_SAXPY) L.A[q_get(wa[u], k)] = op_add<DT>(op_mul<DT>(L.c0, g0[u][k]), g1[u][k]);
+        else if constexpr (OP == JP_OP_PRIV_TMP) {
+          const uint32_t t = op_mul<DT>(L.c0, g0[u][k]);
+          L.T[q_get(xa[u], k)] = t;
+          L.A[q_get(wa[u], k)] = op_add<DT>(t, L.c1);
+        } else L.A[q_get(wa[u], k)] = op_mul<DT>(op_add<DT>(g0[u][k], g1[u][k]), L.c0);
+      }
+    }
+  }
+}
+
 __host__ __device__ static inline bool aligned16(const void *p) { return ((uintptr_t)p & 15) == 0; }
 
 // affine DOALL kernel choice (jp_doall_kernel): 0 LDG/STG.128 grid-stride, 1 bulk-copy (TMA) staged
@@ -196,6 +267,14 @@ static void run_doall(const DLoop &d, cudaStream_t st, int max_ctas) {
     if (max_ctas > 0 && cap > max_ctas) cap = max_ctas;
     int grid = (int)(need < 1 ? 1 : need < cap ? need : cap);
     k_doall_affine_vec<OP, DT><<<grid, kAffThreads, 0, st>>>(d, nvec);
+  } else if (!getenv("JP_DOALL_GENERIC")) {
+    auto al = [](const int32_t *q) { return q == nullptr || ((uintptr_t)q & 15) == 0; };
+    const int vec = al(d.r) && al(d.w) && al(d.r2) && al(d.s);
+    int64_t need = ((d.n + 3) / 4 + 511) / 512;
+    int64_t cap = (int64_t)sms * 8;
+    if (max_ctas > 0 && cap > max_ctas) cap = max_ctas;
+    int grid = (int)(need < 1 ? 1 : need < cap ? need : cap);
+    k_doall_quad<OP, DT><<<grid, 256, 0, st>>>(d, vec);
   } else {
     int64_t need = (d.n + 255) / 256;
     int64_t cap = (int64_t)sms * 8;
