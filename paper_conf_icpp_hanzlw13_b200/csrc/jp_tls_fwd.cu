@@ -418,6 +418,9 @@ cudaError_t tls_fwd_trace_copy(long long *host, int n) {
 #define JP_GRID_K 6
 #endif
 constexpr int kGridT = JP_GRID_T, kGridK = JP_GRID_K;
+#ifndef JP_GRID_EARLY_GATHER
+#define JP_GRID_EARLY_GATHER 0
+#endif
 
 template <int OP, int DT, bool GUIDED, int K>
 struct FwdGrid {
@@ -496,6 +499,13 @@ struct FwdGrid {
     FTR(1);
     fwd_grid_sync(bar, gridDim.x * epoch);
     FTR(2);
+#if JP_GRID_EARLY_GATHER
+    // the next window's gathers right after the barrier, so their latency hides
+    // behind this window's DC / publish / commit; operands this window writes
+    // are stale here and are replaced below by forwarding (a read of an element
+    // written in this window is a raw read, hence probed: q0 / q1)
+    if (more) gather(ws + W, nx, 0);
+#endif
     // ---------------- this window's DC probes and the next window's forwarding
     // probes, all at once; the next window's gathers wait for the end of the
     // window so that probes and polls do not queue behind them ----------------
@@ -596,7 +606,9 @@ struct FwdGrid {
         }
       }
     }
+#if !JP_GRID_EARLY_GATHER
     if (more) gather(ws + W, nx, fwd);
+#endif
     // a second writer of an address in this window (checked last: the log
     // atomics' return values must not hold up the probes issued after the barrier)
 #pragma unroll
