@@ -196,3 +196,25 @@ def test_priv_claim_streams_match_oracle(world, chunk):
     assert reps[0].A.cpu().numpy().tobytes() == A_exp.tobytes()
     st = torch.stack(stats).cpu().numpy()
     assert int(st[:, 0].sum() + st[:, 1].sum()) == n
+
+
+def test_p2p_merge_times_out_instead_of_hanging():
+    """jp_keys_merge_p2p with a peer that never arrives: the device-side barrier
+    gives up after ~4 s and sets the error flag (no hang, no strike)."""
+    import time
+    keys = torch.zeros(1024, dtype=torch.int64, device="cuda")
+    bar = torch.zeros(1, dtype=torch.int64, device="cuda")
+    err = torch.zeros(1, dtype=torch.int32, device="cuda")
+    t0 = time.perf_counter()
+    jp.jp_keys_merge_p2p([keys.data_ptr(), keys.data_ptr()], keys, bar, 1, err)   # world 2, one caller
+    torch.cuda.synchronize()
+    dt = time.perf_counter() - t0
+    assert int(err.item()) == 1 and 3.0 < dt < 30.0, (int(err.item()), dt)
+    # a single-rank merge (world 1) passes both barriers and applies the keys
+    keys[5] = (7 << 32) | 42
+    arr = torch.zeros(1024, dtype=torch.int32, device="cuda")
+    err.zero_()
+    bar.zero_()
+    jp.jp_keys_merge_p2p([keys.data_ptr()], keys, bar, 1, err, arr=arr)
+    torch.cuda.synchronize()
+    assert int(err.item()) == 0 and int(arr[5].item()) == 42 and int(arr.sum().item()) == 42
