@@ -195,11 +195,22 @@ __global__ void __launch_bounds__(256) k_prof_count4(DLoop L, Tabs t, int vec, i
                                                      uint32_t *gsrc) {
   __shared__ unsigned long long s_cnt[3];
   __shared__ unsigned long long s_first;
+  // PRIV_TMP with a small T (config 4: 1024 slots): its first-writer table in
+  // shared memory -- a warp's 32 random slot lookups would otherwise be up to
+  // 32 L1 wavefronts per load
+  __shared__ int32_t s_tT[OP == JP_OP_PRIV_TMP ? kSmemSlots : 1];
   if (threadIdx.x < 3) s_cnt[threadIdx.x] = 0;
   if (threadIdx.x == 0) s_first = ~0ull;
-  JP_CTA_SYNC();
   const int32_t lenA = (int32_t)L.lenA, lenT = (int32_t)L.lenT;
-  const int32_t *rT = OP == JP_OP_PRIV_TMP ? t.wT : t.rT;
+  const int32_t *wT = t.wT;
+  if constexpr (OP == JP_OP_PRIV_TMP) {
+    if (t.wT && lenT <= kSmemSlots) {
+      for (int k = threadIdx.x; k < lenT; k += blockDim.x) s_tT[k] = __ldg(t.wT + k);
+      wT = s_tT;
+    }
+  }
+  JP_CTA_SYNC();
+  const int32_t *rT = OP == JP_OP_PRIV_TMP ? wT : t.rT;
   unsigned c_raw = 0, c_war = 0, c_waw = 0;
   unsigned long long first = ~0ull;
   const int64_t nq = (L.n + 3) >> 2, B = blockDim.x;
@@ -263,7 +274,7 @@ __global__ void __launch_bounds__(256) k_prof_count4(DLoop L, Tabs t, int vec, i
             if (raw) mark_src(a);
           } else if constexpr (OP == JP_OP_PRIV_TMP) {
             war = earlier32(rT, a, lenT, e);
-            waw = earlier32(t.wT, a, lenT, e) || earlier32(t.wA, q4(vb[u], k), lenA, e);
+            waw = earlier32(wT, a, lenT, e) || earlier32(t.wA, q4(vb[u], k), lenA, e);
           } else {
             if constexpr (PAIRS) {
               const int2 pa = pair32(t.pA, a, lenA);
