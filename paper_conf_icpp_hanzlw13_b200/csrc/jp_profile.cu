@@ -516,13 +516,24 @@ static int grid_for(int64_t n, int threads, int per_sm) {
   int64_t cap = (int64_t)num_sms() * per_sm;
   return (int)(need < 1 ? 1 : need < cap ? need : cap);
 }
+// grid-stride kernels with equal work per CTA: one wave of co-resident CTAs
+// (a partial second wave at lower occupancy costs more than it hides)
+static int grid_resident(const void *fn, int64_t n, int threads, size_t smem) {
+  int per = 0;
+  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per, fn, threads, smem) != cudaSuccess || per < 1) {
+    cudaGetLastError();
+    per = 4;
+  }
+  return grid_for(n, threads, per);
+}
 
 template <int OP, int DT>
 static void run_stamp(const DLoop &d, Tabs t, int64_t *hdr, size_t smem, cudaStream_t st) {
   (void)DT;
   if (smem > 48 * 1024) cudaFuncSetAttribute(k_prof_stamp4<OP>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
   const int64_t nq = (d.n + 3) / 4;
-  k_prof_stamp4<OP><<<grid_for((nq + kQuadSteps - 1) / kQuadSteps, 256, 8), 256, smem, st>>>(d, t, idx_vec(d), hdr);
+  k_prof_stamp4<OP><<<grid_resident((const void *)k_prof_stamp4<OP>, (nq + kQuadSteps - 1) / kQuadSteps, 256, smem), 256,
+                      smem, st>>>(d, t, idx_vec(d), hdr);
   note_launch();
 }
 
@@ -602,7 +613,8 @@ static void run_classify(const DLoop &d, Tabs t, uint32_t *bits, int64_t chunk, 
   int64_t tiles = (d.n + 31) / 32;
   if (!bits && !cc) {
     const int64_t nq = (d.n + 3) / 4;
-    k_prof_count4<OP, false><<<grid_for((nq + kQuadSteps - 1) / kQuadSteps, 256, 8), 256, 0, st>>>(d, t, idx_vec(d), hdr,
+    k_prof_count4<OP, false><<<grid_resident((const void *)k_prof_count4<OP, false>, (nq + kQuadSteps - 1) / kQuadSteps,
+                                             256, 0), 256, 0, st>>>(d, t, idx_vec(d), hdr,
                                                                                                  nullptr, nullptr);
   } else {
     k_prof_classify<OP><<<grid_for((tiles + kUnroll - 1) / kUnroll * 32, 256, 8), 256, 0, st>>>(d, t, bits, chunk, cc, hdr,
