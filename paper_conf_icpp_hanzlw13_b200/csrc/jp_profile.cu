@@ -606,6 +606,8 @@ cudaError_t launch_prof_stamp(const Job &j, void *ws, const Layout &lo, cudaStre
   return launch_check();
 }
 
+__global__ void k_interleave(const int32_t *w, const int32_t *r, int2 *pairs, int64_t len);
+
 template <int OP, int DT>
 static void run_classify(const DLoop &d, Tabs t, uint32_t *bits, int64_t chunk, int64_t *cc, int64_t *hdr,
                          uint32_t *src_bits, cudaStream_t st) {
@@ -613,6 +615,16 @@ static void run_classify(const DLoop &d, Tabs t, uint32_t *bits, int64_t chunk, 
   int64_t tiles = (d.n + 31) / 32;
   if (!bits && !cc) {
     const int64_t nq = (d.n + 3) / 4;
+    if constexpr (OP != JP_OP_PRIV_TMP) {
+      if (t.pA) {   // large A tables: classify from interleaved {minW, minR} pairs
+        k_interleave<<<grid_for(d.lenA / 4 + 1, 256, 8), 256, 0, st>>>(t.wA, t.rA, const_cast<int2 *>(t.pA), d.lenA);
+        k_prof_count4<OP, false, true><<<grid_resident((const void *)k_prof_count4<OP, false, true>,
+                                                       (nq + kQuadSteps - 1) / kQuadSteps, 256, 0), 256, 0, st>>>(
+            d, t, idx_vec(d), hdr, nullptr, nullptr);
+        note_launch(2);
+        return;
+      }
+    }
     k_prof_count4<OP, false><<<grid_resident((const void *)k_prof_count4<OP, false>, (nq + kQuadSteps - 1) / kQuadSteps,
                                              256, 0), 256, 0, st>>>(d, t, idx_vec(d), hdr,
                                                                                                  nullptr, nullptr);
@@ -637,6 +649,13 @@ cudaError_t launch_prof_classify(const Job &j, void *ws, const Layout &lo, uint3
     t.as = 2;
   }
   if (src_bits) cudaMemsetAsync(src_bits, 0, 4 * (size_t)((j.d.n + 31) / 32), st);
+  // counts only, separate large A tables: interleave them into the TLS write-log
+  // region (scratch until a TLS run resets it) and classify from the pairs
+  unsigned long long *scratch = at<unsigned long long>(ws, lo, R_TLS_S_A);
+  if (!stamped_pairs && !raw_bits && !chunk_counts && !src_bits && scratch && lo.bytes[R_TLS_S_A] >= 8 * (size_t)j.d.lenA &&
+      t.wA && t.rA && !t.sA && j.d.lenA >= (1 << 20) && ((uintptr_t)t.wA & 15) == 0 && ((uintptr_t)t.rA & 15) == 0 &&
+      getenv_int("JP_CLASSIFY_PAIRS", 1))
+    t.pA = reinterpret_cast<const int2 *>(scratch);
   JP_DISPATCH(j.op, j.dt, run_classify, j.d, t, raw_bits, chunk, chunk_counts, hdr, src_bits, st);
   return launch_check();
 }
