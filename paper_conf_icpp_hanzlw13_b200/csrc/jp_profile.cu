@@ -629,8 +629,8 @@ static void run_classify(const DLoop &d, Tabs t, uint32_t *bits, int64_t chunk, 
                                              256, 0), 256, 0, st>>>(d, t, idx_vec(d), hdr,
                                                                                                  nullptr, nullptr);
   } else {
-    k_prof_classify<OP><<<grid_for((tiles + kUnroll - 1) / kUnroll * 32, 256, 8), 256, 0, st>>>(d, t, bits, chunk, cc, hdr,
-                                                                                                 src_bits);
+    k_prof_classify<OP><<<grid_resident((const void *)k_prof_classify<OP>, (tiles + kUnroll - 1) / kUnroll * 32, 256, 0),
+                          256, 0, st>>>(d, t, bits, chunk, cc, hdr, src_bits);
   }
   note_launch();
 }
