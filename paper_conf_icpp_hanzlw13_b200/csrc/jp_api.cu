@@ -389,6 +389,27 @@ static jp_status static_check(const jp_loop *L, const Job &j, void *ws, const La
   memset(out, 0, sizeof *out);
   int64_t *hdr = at<int64_t>(ws, lo, R_HEADER);
   int *flags = reinterpret_cast<int *>(&hdr[H_AFFINE]);
+  {
+    // a 64-entry prefix of each index array first: an array that is not affine
+    // there is not affine at all, and the full pass (a read of every index
+    // array) is skipped -- the common case of indirect loops
+    constexpr int kS = 64;
+    thread_local int32_t *pin = nullptr;
+    if (!pin && cudaMallocHost(&pin, 4 * kS * sizeof(int32_t)) != cudaSuccess) { pin = nullptr; cudaGetLastError(); }
+    const int32_t *qs[4] = {j.d.r, j.d.r2, j.d.w, j.d.s};
+    const int m = (int)std::min<int64_t>(L->n, kS);
+    if (pin && m >= 3) {
+      for (int q = 0; q < 4; q++)
+        if (qs[q]) JP_CUDA(cudaMemcpyAsync(pin + q * kS, qs[q], 4 * (size_t)m, cudaMemcpyDeviceToHost, st), "affine sample");
+      JP_CUDA(cudaStreamSynchronize(st), "affine sample");
+      for (int q = 0; q < 4; q++) {
+        if (!qs[q]) continue;
+        const int64_t b = pin[q * kS], a = (int64_t)pin[q * kS + 1] - b;
+        for (int k = 2; k < m; k++)
+          if ((int64_t)pin[q * kS + k] != b + a * k) return JP_OK;   // out->affine == 0
+      }
+    }
+  }
   JP_CUDA(launch_affine(j, flags, st), "affine");
   const int32_t *ps[4] = {j.d.r, j.d.r2, j.d.w, j.d.s};
   int32_t first[4][2] = {{0, 0}, {0, 0}, {0, 0}, {0, 0}};
