@@ -190,9 +190,11 @@ __device__ __forceinline__ int2 pair32(const int2 *p, int32_t a, int32_t len) {
   return (uint32_t)a < (uint32_t)len ? __ldg(p + a) : make_int2(-1, -1);
 }
 
+// cc (nullable): per-chunk raw / war / waw counts, chunk % 32 == 0 and >= 128,
+// so a warp's 128 consecutive iterations of one quad step span at most two chunks
 template <int OP, bool GUIDE, bool PAIRS = false>
 __global__ void __launch_bounds__(256) k_prof_count4(DLoop L, Tabs t, int vec, int64_t *hdr, uint32_t *graw,
-                                                     uint32_t *gsrc) {
+                                                     uint32_t *gsrc, int64_t chunk = 0, int64_t *cc = nullptr) {
   __shared__ unsigned long long s_cnt[3];
   __shared__ unsigned long long s_first;
   // PRIV_TMP with a small T (config 4: 1024 slots): its first-writer table in
@@ -238,6 +240,7 @@ __global__ void __launch_bounds__(256) k_prof_count4(DLoop L, Tabs t, int vec, i
     for (int u = 0; u < kQuadSteps; u++) {
       const int64_t q = q0 + u * B;
       uint32_t rb = 0;   // raw bits of this lane's 4 iterations
+      unsigned qr = 0, qa = 0, qw = 0;   // this quad's counts (chunk counts)
       if (q < nq) {
         const int32_t e0 = enc_gid(L.base + (q << 2));
         const int kn = L.n - (q << 2) < 4 ? (int)(L.n - (q << 2)) : 4;
@@ -292,8 +295,25 @@ __global__ void __launch_bounds__(256) k_prof_count4(DLoop L, Tabs t, int vec, i
             if (r1) mark_src(q4(vc[u], k));
           }
           c_raw += raw; c_war += war; c_waw += waw;
+          qr += raw; qa += war; qw += waw;
           rb |= (uint32_t)raw << k;
           if (raw && first == ~0ull) first = (unsigned long long)(L.base + (q << 2) + k);
+        }
+      }
+      if (cc && q0 - threadIdx.x + u * B < nq) {   // warp-uniform: some lane of the warp has a quad
+        const int64_t c = q < nq ? (q << 2) / chunk : -1;
+        const int64_t c0 = __shfl_sync(0xffffffffu, c, 0);
+        const bool in0 = c == c0;
+        const unsigned r0 = __reduce_add_sync(0xffffffffu, in0 ? qr : 0u), r1 = __reduce_add_sync(0xffffffffu, in0 ? 0u : qr);
+        const unsigned a0 = __reduce_add_sync(0xffffffffu, in0 ? qa : 0u), a1 = __reduce_add_sync(0xffffffffu, in0 ? 0u : qa);
+        const unsigned w0 = __reduce_add_sync(0xffffffffu, in0 ? qw : 0u), w1 = __reduce_add_sync(0xffffffffu, in0 ? 0u : qw);
+        const int64_t c1 = __reduce_max_sync(0xffffffffu, (unsigned)(c < 0 ? 0 : c));
+        if ((threadIdx.x & 31) == 0) {
+          auto add = [&](int64_t ch, int kind, unsigned v) {
+            if (v) atomicAdd(reinterpret_cast<unsigned long long *>(&cc[3 * ch + kind]), (unsigned long long)v);
+          };
+          add(c0, 0, r0); add(c0, 1, a0); add(c0, 2, w0);
+          if (c1 != c0) { add(c1, 0, r1); add(c1, 1, a1); add(c1, 2, w1); }
         }
       }
       if constexpr (GUIDE) {
@@ -617,7 +637,8 @@ static void run_classify(const DLoop &d, Tabs t, uint32_t *bits, int64_t chunk, 
     const int64_t nq = (d.n + 3) / 4;
     if constexpr (OP != JP_OP_PRIV_TMP) {
       if (t.pA) {   // large A tables: classify from interleaved {minW, minR} pairs
-        k_interleave<<<grid_for(d.lenA / 4 + 1, 256, 8), 256, 0, st>>>(t.wA, t.rA, const_cast<int2 *>(t.pA), d.lenA);
+        if (t.as == 1)   // (not already stamped as pairs)
+          k_interleave<<<grid_for(d.lenA / 4 + 1, 256, 8), 256, 0, st>>>(t.wA, t.rA, const_cast<int2 *>(t.pA), d.lenA);
         k_prof_count4<OP, false, true><<<grid_resident((const void *)k_prof_count4<OP, false, true>,
                                                        (nq + kQuadSteps - 1) / kQuadSteps, 256, 0), 256, 0, st>>>(
             d, t, idx_vec(d), hdr, nullptr, nullptr);
@@ -628,6 +649,27 @@ static void run_classify(const DLoop &d, Tabs t, uint32_t *bits, int64_t chunk, 
     k_prof_count4<OP, false><<<grid_resident((const void *)k_prof_count4<OP, false>, (nq + kQuadSteps - 1) / kQuadSteps,
                                              256, 0), 256, 0, st>>>(d, t, idx_vec(d), hdr,
                                                                                                  nullptr, nullptr);
+  } else if (cc && chunk >= 128 && (bits == nullptr) == (src_bits == nullptr) &&
+             !(OP == JP_OP_PRIV_TMP && bits) && !getenv("JP_CLASSIFY_BALLOT")) {
+    // chunk counts (and the guide words) from the quad kernel: 4 iterations per
+    // lane, warp-aggregated chunk atomics (the stealing scheduler's profile)
+    const int64_t nq = (d.n + 3) / 4;
+    const int64_t g = (nq + kQuadSteps - 1) / kQuadSteps;
+    if constexpr (OP != JP_OP_PRIV_TMP) {
+      if (bits && t.pA) {
+        k_prof_count4<OP, true, true><<<grid_resident((const void *)k_prof_count4<OP, true, true>, g, 256, 0), 256, 0,
+                                        st>>>(d, t, idx_vec(d), hdr, bits, src_bits, chunk, cc);
+      } else if (bits) {
+        k_prof_count4<OP, true><<<grid_resident((const void *)k_prof_count4<OP, true>, g, 256, 0), 256, 0, st>>>(
+            d, t, idx_vec(d), hdr, bits, src_bits, chunk, cc);
+      } else {
+        k_prof_count4<OP, false><<<grid_resident((const void *)k_prof_count4<OP, false>, g, 256, 0), 256, 0, st>>>(
+            d, t, idx_vec(d), hdr, nullptr, nullptr, chunk, cc);
+      }
+    } else {
+      k_prof_count4<OP, false><<<grid_resident((const void *)k_prof_count4<OP, false>, g, 256, 0), 256, 0, st>>>(
+          d, t, idx_vec(d), hdr, nullptr, nullptr, chunk, cc);
+    }
   } else {
     k_prof_classify<OP><<<grid_resident((const void *)k_prof_classify<OP>, (tiles + kUnroll - 1) / kUnroll * 32, 256, 0),
                           256, 0, st>>>(d, t, bits, chunk, cc, hdr, src_bits);
@@ -647,6 +689,7 @@ cudaError_t launch_prof_classify(const Job &j, void *ws, const Layout &lo, uint3
     t.wA = at<int32_t>(ws, lo, R_TLS_S_A);
     t.rA = t.wA + 1;
     t.as = 2;
+    t.pA = reinterpret_cast<const int2 *>(t.wA);
   }
   if (src_bits) cudaMemsetAsync(src_bits, 0, 4 * (size_t)((j.d.n + 31) / 32), st);
   // counts only, separate large A tables: interleave them into the TLS write-log

@@ -87,17 +87,24 @@ def test_profile_config4_and_5():
     prof_case(synth.config5(n=1 << 16))
 
 
-def test_profile_chunk_counts():
-    wl = synth.config5(n=1 << 16)
+@pytest.mark.parametrize("kernel", ["quad", "ballot"])
+@pytest.mark.parametrize("chunk,n", [(1024, 1 << 16), (160, (1 << 16) + 77), (96, 40000), (32, 5000)])
+def test_profile_chunk_counts(kernel, chunk, n, monkeypatch):
+    """Per-chunk counts (the stealing scheduler's input): the quad kernel with
+    warp-aggregated chunk atomics (chunk >= 128) and the ballot kernel
+    (JP_CLASSIFY_BALLOT=1, and every chunk < 128) against the oracle's flags."""
+    if kernel == "ballot":
+        monkeypatch.setenv("JP_CLASSIFY_BALLOT", "1")
+    wl = synth.config5(n=1 << 16) if n == 1 << 16 else random_loop(n, O.OP_STENCIL2, O.I32, n, len_a=n // 2)
     ref = O.profile(to_oracle(wl))
     g = gpu(wl)
     L = jp.Loop.from_workload(g)
     ws = jp.workspace(L)
-    chunk = 1024
-    cc = torch.full((wl.n // chunk * 3,), -7, dtype=torch.int64, device=DEV)
+    nck = -(-wl.n // chunk)
+    cc = torch.full((nck * 3,), -7, dtype=torch.int64, device=DEV)
     jp.jp_profile_density(L, ws, chunk_iters=chunk, chunk_counts=cc)
     cc = cc.cpu().numpy().reshape(-1, 3)
-    f = ref["flags"].reshape(-1, chunk)
+    f = np.concatenate([ref["flags"], np.zeros(nck * chunk - wl.n, dtype=ref["flags"].dtype)]).reshape(-1, chunk)
     assert np.array_equal(cc[:, 0], (f & 1).sum(1))
     assert np.array_equal(cc[:, 1], ((f >> 1) & 1).sum(1))
     assert np.array_equal(cc[:, 2], ((f >> 2) & 1).sum(1))
