@@ -649,7 +649,7 @@ static int64_t auto_w_max(const jp_profile *p) {
 // workspace allow it (jp_schedule)
 static jp_status run_tls_job(const jp_loop *L, const Job &j, const jp_tls_cfg *cfg, const jp_profile *prof, void *ws,
                              size_t ws_bytes, jp_tls_stats *stats, cudaStream_t st, bool auto_guide = false,
-                             TlsPlan *plan_out = nullptr, bool guide_ready = false, bool s_clean = false) {
+                             TlsPlan *plan_out = nullptr, bool guide_ready = false, int s_clean = 0) {
   TlsPlan tp;
   JP_TRY(tls_plan(j, cfg, prof, tp));
   const bool helps = tp.path == 3 || tp.path >= 5 || (tp.path == 1 && prof && prof->n > 0 && prof->raw_iters * 50 <= prof->n);
@@ -1003,7 +1003,7 @@ static Job sub_job(const Job &j, int64_t s, int64_t e) {
 
 static jp_status run_mode(const jp_loop *L, const Job &j, int mode, const jp_profile *prof, const jp_sched_cfg &c,
                           void *ws, size_t ws_bytes, jp_sched_result *res, cudaStream_t st, bool guide_ready = false,
-                          bool s_clean = false) {
+                          int s_clean = 0) {
   Layout lo = layout(L);
   if (mode == JP_MODE_DOALL) {
     JP_CUDA(launch_doall(j, st), "doall");
@@ -1483,13 +1483,32 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
   const Layout lg = layout(L);
   const bool gfuse = lg.bytes[R_GUIDE] && ws && ws_bytes >= layout_end(lg, JP_WS_PROFILE | JP_WS_GUIDE | JP_WS_TLS);
   bool pairs = false;
+  int clean = 0;
+  cudaEvent_t vdone = nullptr;
   if (gfuse) {
     // large A tables: stamped straight into {minW, minR} pairs (one 8-byte entry
     // per address for the classify lookups; the separate tables stay unwritten)
     pairs = stamp_pairs_ok(j, ws, lg);
+    // the on-chip TLS shadow values must start at zero: clear them on a side
+    // stream while the (L2-atomic-bound) profile runs, instead of after it
+    auto *V = at<unsigned long long>(ws, lg, R_TLS_C_A);
+    if (pairs && V && cudaEventCreateWithFlags(&vdone, cudaEventDisableTiming) == cudaSuccess) {
+      cudaStream_t side = g_pool.get(40);
+      cudaEventRecord(vdone, st);          // after whatever ran before on st
+      cudaStreamWaitEvent(side, vdone, 0);
+      cudaMemsetAsync(V, 0, lg.bytes[R_TLS_C_A], side);
+      cudaEventRecord(vdone, side);
+      clean = 2;
+    }
+    if (pairs) clean |= 1;
     if (pairs) JP_CUDA(launch_prof_stamp(j, ws, lg, st, true), "profile stamp");
     else JP_TRY(jp_profile_stamp(L, ws, ws_bytes, stp));
     JP_CUDA(launch_prof_classify_guide(j, ws, lg, st, pairs), "profile classify");
+    if (vdone) {   // everything after the profile on st (TLS, or any later call) sees V zeroed
+      cudaStreamWaitEvent(st, vdone, 0);
+      cudaEventDestroy(vdone);
+      vdone = nullptr;
+    }
     int64_t h[8];
     JP_CUDA(d2h_small_sync(h, at<int64_t>(ws, lg, R_HEADER), sizeof h, st), "profile D2H");
     if (h[H_BAD]) return fail(JP_ERR_INDEX, "%lld index entries are outside their arrays", (long long)h[H_BAD]);
@@ -1502,7 +1521,7 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
   res->mode = select_mode_counts(p.n, p.raw_iters, p.war_iters, p.waw_iters, c.tau_high);
   res->n_tasks = 1;
   res->n_batches = 1;
-  return run_mode(L, j, res->mode, &p, c, ws, ws_bytes, res, st, gfuse && p.waw_iters == 0, pairs);
+  return run_mode(L, j, res->mode, &p, c, ws, ws_bytes, res, st, gfuse && p.waw_iters == 0, clean);
 }
 
 

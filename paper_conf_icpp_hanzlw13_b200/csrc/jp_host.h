@@ -130,7 +130,7 @@ int tls_fwd_max_cluster();           // 16 when the device schedules it, else 8
 cudaError_t launch_tls_fwd_grid(const Job &j, int64_t window, const uint32_t *bits, const uint32_t *bsrc,
                                 unsigned long long *S,
                                 unsigned long long *V, int64_t lenS, unsigned *bar, int64_t *stats,
-                                cudaStream_t st, bool s_clean = false);
+                                cudaStream_t st, int clean = 0);   // bit 0: S clean, bit 1: V zeroed
 int64_t tls_fwd_grid_wcap();         // slots per CTA * co-resident CTAs (2048 * 148 on B200)
 int64_t tls_fwd_grid_cta_slots();    // window iterations per CTA of the all-SM kernel
 // stats: int64[4] device (committed, executed, windows, violations); bar: u32[2]

@@ -677,17 +677,18 @@ static void run_fwd_grid(cudaError_t &e, const Job &j, uint32_t W, const uint32_
 cudaError_t launch_tls_fwd_grid(const Job &j, int64_t window, const uint32_t *bits, const uint32_t *bsrc,
                                 unsigned long long *S,
                                 unsigned long long *V, int64_t lenS, unsigned *bar, int64_t *stats,
-                                cudaStream_t st, bool s_clean) {
+                                cudaStream_t st, int clean) {
   if (j.d.n == 0) {
     cudaMemsetAsync(stats, 0, 4 * sizeof(int64_t), st);
     return launch_check();
   }
   if (S && lenS > 0) {   // epoch 0: no writer yet
-    // s_clean: S holds this call's {minW, minR} stamp pairs, whose high words
+    // clean bit 0: S holds this call's {minW, minR} stamp pairs, whose high words
     // (encoded gids >= 2^31 - 2^24, or all ones) never equal a window epoch
     // (< 2^24): they already read as "no writer this window"
-    if (!s_clean) cudaMemsetAsync(S, 0, 8 * (size_t)lenS, st);
-    cudaMemsetAsync(V, 0, 8 * (size_t)lenS, st);
+    // clean bit 1: the caller already zeroed V (on a side stream, behind the profile)
+    if (!(clean & 1)) cudaMemsetAsync(S, 0, 8 * (size_t)lenS, st);
+    if (!(clean & 2)) cudaMemsetAsync(V, 0, 8 * (size_t)lenS, st);
   }
   cudaMemsetAsync(bar, 0, 2 * sizeof(unsigned), st);
   cudaMemsetAsync(stats, 0, 4 * sizeof(int64_t), st);
