@@ -1461,34 +1461,55 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
     }
     return JP_OK;
   }
+  // the pair table of the profile (all ones = no stamp yet) is filled on a side
+  // stream from the start, overlapping the static check's prefix read
+  const Layout lg = layout(L);
+  const bool gfuse = lg.bytes[R_GUIDE] && ws && ws_bytes >= layout_end(lg, JP_WS_PROFILE | JP_WS_GUIDE | JP_WS_TLS);
+  const bool pairs = gfuse && stamp_pairs_ok(j, ws, lg);
+  cudaEvent_t pdone = nullptr;
+  if (pairs && cudaEventCreateWithFlags(&pdone, cudaEventDisableTiming) == cudaSuccess) {
+    cudaStream_t side = g_pool.get(41);
+    cudaEventRecord(pdone, st);
+    cudaStreamWaitEvent(side, pdone, 0);
+    cudaMemsetAsync(at<char>(ws, lg, R_TLS_S_A), 0xFF, 8 * (size_t)L->len_A, side);
+    cudaEventRecord(pdone, side);
+  }
+  // st waits for the fill before its next use of the region (the stamp, or the
+  // DOALL exit below): every path after this point calls it once
+  auto join_fill = [&]() {
+    if (pdone) {
+      cudaStreamWaitEvent(st, pdone, 0);
+      cudaEventDestroy(pdone);
+      pdone = nullptr;
+    }
+  };
+  const bool pairs_ready = pdone != nullptr;
   if (c.static_check == 0 && ws) {
     // static analysis lite: affine, in-range, conflict-free -> DOALL without a profile
     Layout ls;
-    JP_TRY(check_ws(L, ws, ws_bytes, 0, ls));
+    if (jp_status e0 = check_ws(L, ws, ws_bytes, 0, ls)) { join_fill(); return e0; }
     jp_static sa;
-    JP_TRY(static_check(L, j, ws, ls, &sa, st));
+    if (jp_status e1 = static_check(L, j, ws, ls, &sa, st)) { join_fill(); return e1; }
     if (sa.independent && sa.in_range) {
       res->mode = JP_MODE_DOALL;
       res->profiled = 0;
       res->n_tasks = 1;
       res->n_batches = 1;
+      join_fill();
       JP_CUDA(launch_doall(j, st), "doall");
       res->task_mode_iters[JP_MODE_DOALL] = L->n;
       return JP_OK;
     }
   }
+  join_fill();
   jp_profile p;
   // the classify pass also writes the TLS guide bitmaps when the loop can be guided
   // (A read through an index, workspace with the guide region): no separate guide pass
-  const Layout lg = layout(L);
-  const bool gfuse = lg.bytes[R_GUIDE] && ws && ws_bytes >= layout_end(lg, JP_WS_PROFILE | JP_WS_GUIDE | JP_WS_TLS);
-  bool pairs = false;
   int clean = 0;
   cudaEvent_t vdone = nullptr;
   if (gfuse) {
     // large A tables: stamped straight into {minW, minR} pairs (one 8-byte entry
     // per address for the classify lookups; the separate tables stay unwritten)
-    pairs = stamp_pairs_ok(j, ws, lg);
     // the on-chip TLS shadow values must start at zero: clear them on a side
     // stream while the (L2-atomic-bound) profile runs, instead of after it
     auto *V = at<unsigned long long>(ws, lg, R_TLS_C_A);
@@ -1501,7 +1522,7 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
       clean = 2;
     }
     if (pairs) clean |= 1;
-    if (pairs) JP_CUDA(launch_prof_stamp(j, ws, lg, st, true), "profile stamp");
+    if (pairs) JP_CUDA(launch_prof_stamp(j, ws, lg, st, true, pairs_ready), "profile stamp");
     else JP_TRY(jp_profile_stamp(L, ws, ws_bytes, stp));
     JP_CUDA(launch_prof_classify_guide(j, ws, lg, st, pairs), "profile classify");
     if (vdone) {   // everything after the profile on st (TLS, or any later call) sees V zeroed

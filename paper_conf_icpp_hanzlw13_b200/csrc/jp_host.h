@@ -48,7 +48,8 @@ cudaError_t launch_validate(const Job &j, int64_t *hdr, cudaStream_t st);
 // stamp tables of a profile on the same workspace; no sync.
 cudaError_t launch_tls_guide(const Job &j, void *ws, const Layout &lo, cudaStream_t st);
 // pairs: stamp the A tables into interleaved {minW, minR} pairs in region 7 (see stamp_pairs_ok)
-cudaError_t launch_prof_stamp(const Job &j, void *ws, const Layout &lo, cudaStream_t st, bool pairs = false);
+cudaError_t launch_prof_stamp(const Job &j, void *ws, const Layout &lo, cudaStream_t st, bool pairs = false,
+                              bool pairs_ready = false);
 bool stamp_pairs_ok(const Job &j, void *ws, const Layout &lo);
 // src_bits (nullable): also the TLS guide's RAW-source words (raw_bits then holds its raw words)
 cudaError_t launch_prof_classify(const Job &j, void *ws, const Layout &lo, uint32_t *raw_bits,

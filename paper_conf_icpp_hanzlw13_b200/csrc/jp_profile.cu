@@ -584,7 +584,7 @@ bool stamp_pairs_ok(const Job &j, void *ws, const Layout &lo) {
          (lo.off[R_TLS_S_A] & 15) == 0 && ws;
 }
 
-cudaError_t launch_prof_stamp(const Job &j, void *ws, const Layout &lo, cudaStream_t st, bool pairs) {
+cudaError_t launch_prof_stamp(const Job &j, void *ws, const Layout &lo, cudaStream_t st, bool pairs, bool pairs_ready) {
   int64_t *hdr = at<int64_t>(ws, lo, R_HEADER);
   cudaMemsetAsync(hdr, 0, kHeaderBytes, st);
   cudaMemsetAsync(&hdr[H_FIRST_RAW], 0xFF, sizeof(int64_t), st);   // none (= ~0 for the u64 atomicMin)
@@ -596,7 +596,7 @@ cudaError_t launch_prof_stamp(const Job &j, void *ws, const Layout &lo, cudaStre
   }
   int32_t *pw = pairs ? at<int32_t>(ws, lo, R_TLS_S_A) : nullptr;
   if (pw) {
-    cudaMemsetAsync(pw, 0xFF, 8 * (size_t)j.d.lenA, st);
+    if (!pairs_ready) cudaMemsetAsync(pw, 0xFF, 8 * (size_t)j.d.lenA, st);   // (else filled by the caller)
     tab_bytes += 8 * (size_t)j.d.lenA;
   }
   if (j.d.n == 0) return launch_check();
