@@ -1148,6 +1148,9 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
   uint32_t *gbits = gfuse ? at<uint32_t>(ws, lo, R_GUIDE) : nullptr;
   // large A tables: stamped as {minW, minR} pairs in region 7 (free until the TLS tasks run)
   const bool pairs = stamp_pairs_ok(j, ws, lo);
+  // the first all-SM TLS task finds this call's pair table in the write-log
+  // region: it needs no reset (see launch_tls_fwd_grid); later ones do
+  bool s_fresh = pairs;
   JP_CUDA(launch_prof_stamp(j, ws, lo, st, pairs), "profile stamp");
   JP_CUDA(launch_prof_classify(j, ws, lo, gbits, chunk, cc, st, gbits ? gbits + (L->n + 31) / 32 : nullptr, pairs),
           "profile classify");
@@ -1285,8 +1288,9 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
         JP_CUDA(launch_tls_fwd_grid(sj, tp.window, b0, b1, at<unsigned long long>(ws, lo, R_TLS_S_A),
                                     at<unsigned long long>(ws, lo, R_TLS_C_A), L->len_A,
                                     reinterpret_cast<unsigned *>(&at<int64_t>(ws, lo, R_HEADER)[H_BAR_COUNT]),
-                                    tstats + 4 * t, st),
+                                    tstats + 4 * t, st, s_fresh ? 1 : 0),
                 "tls task");
+        s_fresh = false;
       } else {
         JP_CUDA(launch_tls_fwd(sj, tp.window, tp.cluster, b0, b1, tstats + 4 * t, st), "tls task");
       }

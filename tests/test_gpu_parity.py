@@ -975,3 +975,33 @@ def test_memcheck_clean():
                           os.path.join(root, "scripts", "sanitize.py")], capture_output=True, text=True, timeout=900)
     assert "DONE fails=0" in out.stdout, out.stdout[-2000:] + out.stderr[-2000:]
     assert "ERROR SUMMARY: 0 errors" in out.stdout + out.stderr, out.stdout[-2000:]
+
+
+def test_schedule_stealing_two_grid_tls_tasks():
+    """Two TLS regions (each beyond a 16-CTA cluster: the all-SM on-chip path)
+    separated by DOALL regions, all on disjoint addresses: one batch whose two
+    grid TLS tasks run back to back -- the first reuses the profile's pair table
+    as its clean write log, the second must reset it."""
+    m = 1 << 16
+    parts_r, parts_w = [], []
+    g = np.random.default_rng(4)
+    for k in range(4):
+        base = k * m
+        if k % 2 == 0:
+            p = torch.from_numpy((g.permutation(m) + base).astype(np.int32))
+            parts_r.append(p)
+            parts_w.append(p.clone())
+        else:
+            r, w, _ = synth.gen.dep_region(1100 + k, m, base, 0.05, 512)
+            parts_r.append(r)
+            parts_w.append(w)
+    n = 4 * m
+    A = torch.from_numpy(g.integers(0, 1 << 20, size=n).astype(np.int32))
+    wl = synth.Workload("two_tls", O.OP_ADD_C, O.I32, n, A, r=torch.cat(parts_r), w=torch.cat(parts_w), c0=7)
+    _, Aexp, _ = O.run_seq(to_oracle(wl))
+    gw = gpu(wl)
+    L = jp.Loop.from_workload(gw)
+    res = jp.jp_schedule(L, jp.workspace(L), scheme=jp.JP_SCHED_STEALING, chunk_iters=4096)
+    torch.cuda.synchronize()
+    check_arrays(gw, Aexp, None)
+    assert res["n_tasks"] == 4 and res["task_mode_iters"][jp.JP_MODE_TLS] == 2 * m and res["tls_path"] == 6, res
