@@ -278,8 +278,18 @@ def _res_dict(r: _abi.jp_sched_result) -> dict:
             "tls_w_max": wmax, "tls_path": path, "tls_guided": guided, "tls_recovery": rec, "tls_cluster": cl}
 
 
+_DEFAULT_CFG = None
+
+
 def jp_schedule(loop: Loop, ws=None, cfg=None, stream=None, **kw) -> dict:
-    cfg = cfg if cfg is not None else sched_cfg(**kw)
+    global _DEFAULT_CFG
+    if cfg is None:
+        if kw:
+            cfg = sched_cfg(**kw)
+        else:   # the C call only reads it (const jp_sched_cfg *): one shared default
+            if _DEFAULT_CFG is None:
+                _DEFAULT_CFG = sched_cfg()
+            cfg = _DEFAULT_CFG
     res = _abi.jp_sched_result()
     p, nb = _ws(ws)
     check(lib().jp_schedule(loop.ref, C.byref(cfg), p, nb, C.byref(res), _stream(stream)))
