@@ -691,6 +691,25 @@ def run_jp(args):
            "h2d_bytes_per_step": int(sum_over_ranks(8 * (s1 - s0), world, dev)),
            "d2h_bytes_per_step": int(sum_over_ranks(4 * (s1 - s0), world, dev)),
            "api": "jp_schedule_host (pinned host X,Y -> H2D -> DOALL -> D2H Y)"}
+    # the copy-only bound of the same step: X, Y up and Y down on two streams, no kernel
+    dX = stage[:4 * (s1 - s0)].view(torch.float32)
+    dY = stage[4 * (s1 - s0):8 * (s1 - s0)].view(torch.float32)
+    su, sd = torch.cuda.Stream(), torch.cuda.Stream()
+
+    def copies():
+        with torch.cuda.stream(su):
+            dX.copy_(hX, non_blocking=True)
+            dY.copy_(hA, non_blocking=True)
+        with torch.cuda.stream(sd):
+            hA.copy_(dY, non_blocking=True)
+    copies()
+    torch.cuda.synchronize()
+    tc = time.perf_counter()
+    copies()
+    torch.cuda.synchronize()
+    tc = max_over_ranks(time.perf_counter() - tc, world, dev)
+    e2e["pcie_copy_only_bound"] = N2 / tc
+    e2e["frac_of_copy_bound"] = e2e["value"] / (N2 / tc)
     del stage, hA, hX
     launches_all = int(sum_over_ranks(launches, world, dev))
 
