@@ -677,6 +677,36 @@ static void run_classify(const DLoop &d, Tabs t, uint32_t *bits, int64_t chunk, 
   note_launch();
 }
 
+// PRIV_TMP with identity Y writes and an indirect scratch index s: no exposed
+// read of a written array (X is read-only, T's read is covered), so raw = 0,
+// and war_i = waw_i = "an earlier iteration wrote T[s_i]" = "i is not the first
+// writer of its slot".  Every slot whose (global) first writer lies in this
+// range has exactly one such iteration, so war = waw = n - #{slots whose first
+// writer is in [base, base + n)}: one pass over the small T table replaces the
+// classify pass over the s stream.
+__global__ void __launch_bounds__(1024) k_slot_first_writers(const int32_t *wT, int64_t lenT, int64_t base, int64_t n,
+                                                             int64_t *hdr) {
+  __shared__ unsigned long long cnt;
+  if (threadIdx.x == 0) cnt = 0;
+  __syncthreads();
+  unsigned c = 0;
+  for (int64_t a = threadIdx.x; a < lenT; a += blockDim.x) {
+    const int32_t v = wT[a];
+    if (v >= 0) {
+      const int64_t gid = 0x7FFFFFFF - (int64_t)v;
+      c += gid >= base && gid < base + n;
+    }
+  }
+  c = __reduce_add_sync(0xffffffffu, c);
+  if ((threadIdx.x & 31) == 0 && c) atomicAdd(&cnt, (unsigned long long)c);
+  __syncthreads();
+  if (threadIdx.x == 0) {
+    hdr[H_RAW] = 0;
+    hdr[H_WAR] = n - (int64_t)cnt;
+    hdr[H_WAW] = n - (int64_t)cnt;
+  }
+}
+
 cudaError_t launch_prof_classify(const Job &j, void *ws, const Layout &lo, uint32_t *raw_bits, int64_t chunk,
                                  int64_t *chunk_counts, cudaStream_t st, uint32_t *src_bits, bool stamped_pairs) {
   int64_t *hdr = at<int64_t>(ws, lo, R_HEADER);
@@ -685,6 +715,12 @@ cudaError_t launch_prof_classify(const Job &j, void *ws, const Layout &lo, uint3
   if (chunk_counts) cudaMemsetAsync(chunk_counts, 0, sizeof(int64_t) * 3 * ((j.d.n + chunk - 1) / chunk), st);
   if (j.d.n == 0) return launch_check();
   Tabs t = tabs_of(j.d, ws, lo);
+  if (j.op == JP_OP_PRIV_TMP && !j.d.w && j.d.s && t.wT && !raw_bits && !chunk_counts && !src_bits &&
+      !getenv("JP_CLASSIFY_FULL")) {
+    k_slot_first_writers<<<1, 1024, 0, st>>>(t.wT, j.d.lenT, j.d.base, j.d.n, hdr);
+    note_launch();
+    return launch_check();
+  }
   if (stamped_pairs) {   // the stamp pass wrote {minW, minR} pairs into region 7
     t.wA = at<int32_t>(ws, lo, R_TLS_S_A);
     t.rA = t.wA + 1;

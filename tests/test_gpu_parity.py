@@ -1005,3 +1005,32 @@ def test_schedule_stealing_two_grid_tls_tasks():
     torch.cuda.synchronize()
     check_arrays(gw, Aexp, None)
     assert res["n_tasks"] == 4 and res["task_mode_iters"][jp.JP_MODE_TLS] == 2 * m and res["tls_path"] == 6, res
+
+
+@pytest.mark.parametrize("full", ["0", "1"])
+@pytest.mark.parametrize("seed,n,slots", [(1, 5000, 64), (2, 70001, 1024), (3, 100, 4096), (4, 300000, 8192)])
+def test_priv_tmp_slot_count_profile(seed, n, slots, full, monkeypatch):
+    """PRIV_TMP with identity Y: war = waw = n - #slots first-written in the range,
+    from the T table alone (JP_CLASSIFY_FULL=1: the classify pass) -- both equal
+    the oracle, for the whole loop and for a range of it."""
+    if full == "1":
+        monkeypatch.setenv("JP_CLASSIFY_FULL", "1")
+    g = np.random.default_rng(seed)
+    wl = synth.Workload("pt", O.OP_PRIV_TMP, O.F32, n, torch.from_numpy(g.standard_normal(n).astype(np.float32)),
+                        s=torch.from_numpy(g.integers(0, slots, size=n).astype(np.int32)),
+                        X=torch.from_numpy(g.standard_normal(n).astype(np.float32)),
+                        T=torch.from_numpy(g.standard_normal(slots).astype(np.float32)), c0=1.1, c1=0.3)
+    ref = O.profile(to_oracle(wl))
+    gw = gpu(wl)
+    L = jp.Loop.from_workload(gw)
+    p = jp.jp_profile_density(L, jp.workspace(L))
+    assert (p["raw_iters"], p["war_iters"], p["waw_iters"], p["first_raw_iter"]) == \
+        (ref["raw_iters"], ref["war_iters"], ref["waw_iters"], -1)
+    # a range [b, e) of the loop (stamped alone: its own first writers)
+    b, e = n // 3, n - n // 5
+    sub = synth.Workload("pt_sub", O.OP_PRIV_TMP, O.F32, e - b, wl.A[b:e].clone(), s=wl.s[b:e].clone(),
+                         X=wl.X[b:e].clone(), T=wl.T.clone(), c0=1.1, c1=0.3)
+    rs = O.profile(to_oracle(sub))
+    Ls = jp.Loop.from_workload(gpu(sub))
+    ps = jp.jp_profile_density(Ls, jp.workspace(Ls))
+    assert (ps["war_iters"], ps["waw_iters"]) == (rs["war_iters"], rs["waw_iters"])
