@@ -298,6 +298,14 @@ jp_status jp_priv_finalize(const jp_loop *L, void *ws, size_t ws_bytes, jp_strea
  * the same first violators.  Needs JP_WS_PROFILE | JP_WS_GUIDE.  No sync.
  * Loops whose A is not reached through an index have no guide (no-op).     */
 jp_status jp_tls_guide(const jp_loop *L, void *ws, size_t ws_bytes, jp_stream_t st);
+/* Reading A8's adaptive window policy ("sub-loops" of unspecified
+ * size), the same function every TLS kernel applies:
+ *   prev_commit < 0 (first window): prof_raw_iters < 0 (no profile) -> 4096,
+ *     == 0 -> w_max, else pow2ceil(ceil(4n / prof_raw_iters));
+ *   after a window that committed c iterations: pow2ceil(2 * max(c, 16));
+ * both clamped to [32, w_max].  Host only, no device needed; returns -1 when
+ * n < 0 or w_max < 32.                                                       */
+int64_t jp_tls_next_window(int64_t n, int64_t prof_raw_iters, int64_t prev_commit, int64_t w_max);
 jp_status jp_run_tls(const jp_loop *L, const jp_tls_cfg *cfg /* host */, const jp_profile *prof,
                      void *ws, size_t ws_bytes, jp_tls_stats *stats, jp_stream_t st);
 

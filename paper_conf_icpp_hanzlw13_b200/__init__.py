@@ -24,7 +24,7 @@ from ._abi import (  # noqa: F401
 __all__ = [
     "Loop", "workspace", "jp_workspace_bytes", "jp_ws_region", "jp_validate", "jp_profile_stamp",
     "jp_profile_classify", "jp_profile_density", "jp_select_mode", "jp_run_doall", "jp_run_privatized",
-    "jp_priv_stream", "jp_priv_finalize", "jp_doall_kernel", "jp_tls_guide", "tls_first_window", "jp_run_tls", "jp_schedule", "jp_stage_bytes", "jp_schedule_host",
+    "jp_priv_stream", "jp_priv_finalize", "jp_doall_kernel", "jp_tls_guide", "jp_tls_next_window", "jp_run_tls", "jp_schedule", "jp_stage_bytes", "jp_schedule_host",
     "jp_plan_sharing", "jp_plan_stealing", "jp_merge_apply",
     "jp_plan", "jp_plan_tasks", "jp_export_keys", "jp_keys_merge_p2p", "jp_run_priv_claim", "jp_run_doall_spill", "jp_ipc_export", "jp_ipc_import", "jp_ipc_close",
     "jp_sparse_scratch_bytes", "jp_sparse_pack", "jp_sparse_reduce_max", "jp_sparse_gather", "jp_sparse_scatter",
@@ -224,17 +224,9 @@ def jp_doall_kernel(which: int = -1) -> int:
     return int(lib().jp_doall_kernel(int(which)))
 
 
-def tls_first_window(n: int, raw_iters: int, w_max: int = 4096) -> int:
-    """Reading A8's first adaptive window (jp.h): clamp(pow2ceil(ceil(4n/raw)), 32, w_max),
-    w_max when raw == 0, 4096 without a profile (raw < 0).  Host arithmetic only."""
-    if raw_iters < 0:
-        w0 = 4096
-    elif raw_iters == 0:
-        w0 = w_max
-    else:
-        q = (4 * n + raw_iters - 1) // raw_iters
-        w0 = 1 << max(0, (q - 1).bit_length())
-    return max(32, min(w0, w_max))
+def jp_tls_next_window(n: int, prof_raw_iters: int, prev_commit: int = -1, w_max: int = 4096) -> int:
+    """Reading A8's window policy, computed by the library (jp.h)."""
+    return int(lib().jp_tls_next_window(int(n), int(prof_raw_iters), int(prev_commit), int(w_max)))
 
 
 def jp_tls_guide(loop: Loop, ws: torch.Tensor, stream=None) -> None:

@@ -101,6 +101,7 @@ SIGNATURES = [
     ("jp_priv_finalize", _I32, [_P(jp_loop), _V, _SZ, _V]),
     ("jp_doall_kernel", _I32, [_I32]),
     ("jp_tls_guide", _I32, [_P(jp_loop), _V, _SZ, _V]),
+    ("jp_tls_next_window", _I64, [_I64, _I64, _I64, _I64]),
     ("jp_run_tls", _I32, [_P(jp_loop), _P(jp_tls_cfg), _P(jp_profile), _V, _SZ, _P(jp_tls_stats), _V]),
     ("jp_schedule", _I32, [_P(jp_loop), _P(jp_sched_cfg), _V, _SZ, _P(jp_sched_result), _V]),
     ("jp_stage_bytes", _SZ, [_P(jp_loop)]),

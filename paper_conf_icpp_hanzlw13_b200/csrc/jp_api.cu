@@ -460,6 +460,11 @@ static jp_status static_check(const jp_loop *L, const Job &j, void *ws, const La
   return JP_OK;
 }
 
+int64_t jp_tls_next_window(int64_t n, int64_t prof_raw_iters, int64_t prev_commit, int64_t w_max) {
+  if (n < 0 || w_max < 32) return -1;
+  return tls_next_window(n, prof_raw_iters, prev_commit, w_max);
+}
+
 int32_t jp_affine_dependence(int64_t af, int64_t bf, int64_t ag, int64_t bg, int64_t n) {
   return affine_conflict(af, bf, ag, bg, n) ? 1 : 0;
 }
@@ -1511,6 +1516,13 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
   // (A read through an index, workspace with the guide region): no separate guide pass
   int clean = 0;
   cudaEvent_t vdone = nullptr;
+  // every exit (an error return included) orders st after the side-stream clear
+  // of the shadow values and releases the event
+  struct JoinV {
+    cudaEvent_t &e; cudaStream_t s;
+    void join() { if (e) { cudaStreamWaitEvent(s, e, 0); cudaEventDestroy(e); e = nullptr; } }
+    ~JoinV() { join(); }
+  } join_v{vdone, st};
   if (gfuse) {
     // large A tables: stamped straight into {minW, minR} pairs (one 8-byte entry
     // per address for the classify lookups; the separate tables stay unwritten)
@@ -1529,11 +1541,7 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
     if (pairs) JP_CUDA(launch_prof_stamp(j, ws, lg, st, true, pairs_ready), "profile stamp");
     else JP_TRY(jp_profile_stamp(L, ws, ws_bytes, stp));
     JP_CUDA(launch_prof_classify_guide(j, ws, lg, st, pairs), "profile classify");
-    if (vdone) {   // everything after the profile on st (TLS, or any later call) sees V zeroed
-      cudaStreamWaitEvent(st, vdone, 0);
-      cudaEventDestroy(vdone);
-      vdone = nullptr;
-    }
+    join_v.join();   // everything after the profile on st (TLS, or any later call) sees V zeroed
     int64_t h[8];
     JP_CUDA(d2h_small_sync(h, at<int64_t>(ws, lg, R_HEADER), sizeof h, st), "profile D2H");
     if (h[H_BAD]) return fail(JP_ERR_INDEX, "%lld index entries are outside their arrays", (long long)h[H_BAD]);

@@ -707,6 +707,8 @@ __global__ void __launch_bounds__(1024) k_slot_first_writers(const int32_t *wT, 
   }
 }
 
+static constexpr int64_t kSlotCountMaxT = 1 << 20;
+
 cudaError_t launch_prof_classify(const Job &j, void *ws, const Layout &lo, uint32_t *raw_bits, int64_t chunk,
                                  int64_t *chunk_counts, cudaStream_t st, uint32_t *src_bits, bool stamped_pairs) {
   int64_t *hdr = at<int64_t>(ws, lo, R_HEADER);
@@ -715,8 +717,10 @@ cudaError_t launch_prof_classify(const Job &j, void *ws, const Layout &lo, uint3
   if (chunk_counts) cudaMemsetAsync(chunk_counts, 0, sizeof(int64_t) * 3 * ((j.d.n + chunk - 1) / chunk), st);
   if (j.d.n == 0) return launch_check();
   Tabs t = tabs_of(j.d, ws, lo);
+  // the one-CTA slot count reads all of T's table: taken only when that table is
+  // small next to the s stream the full pass would read (config 4: 1024 slots)
   if (j.op == JP_OP_PRIV_TMP && !j.d.w && j.d.s && t.wT && !raw_bits && !chunk_counts && !src_bits &&
-      !getenv("JP_CLASSIFY_FULL")) {
+      j.d.lenT <= kSlotCountMaxT && j.d.lenT <= j.d.n / 8 + 1024 && !getenv("JP_CLASSIFY_FULL")) {
     k_slot_first_writers<<<1, 1024, 0, st>>>(t.wT, j.d.lenT, j.d.base, j.d.n, hdr);
     note_launch();
     return launch_check();

@@ -160,9 +160,16 @@ class P2PMerge:
         torch.cuda.synchronize()
         dist.barrier(group=group)
 
-    def run(self, arr=None, stream=None):
+    def run(self, table=None, arr=None, stream=None):
+        """Merge (and apply to ``arr``).  Raises if the device barrier timed out:
+        the keys are then NOT merged and nothing was applied on this rank."""
+        if table is not None and (table.data_ptr() != self.table.data_ptr() or table.numel() != self.table.numel()):
+            raise ValueError("P2PMerge.run: this handle maps a different key table")
         self.epoch += 1
         self.jp.jp_keys_merge_p2p(self.ptrs, self.table, self.bar_ref, self.epoch, self.err, arr, stream)
+        if not self.ok():
+            raise RuntimeError(f"p2p key merge (epoch {self.epoch}): device barrier timed out on rank {self.rank}; "
+                               "keys not merged")
 
     def ok(self) -> bool:
         return int(self.err.item()) == 0
@@ -173,14 +180,19 @@ class P2PMerge:
         self._opened = []
 
 
-_P2P = {}
-
-
-def _p2p_for(t, group):
-    key = (t.data_ptr(), t.numel(), id(group))
-    if key not in _P2P:
-        _P2P[key] = P2PMerge(t, group)
-    return _P2P[key]
+def p2p_handles(loop, ws, group=None, engine=None) -> dict:
+    """Collective: one P2PMerge per small key table of ``loop`` in ``ws`` (every
+    rank must call it with its own replica).  The handles keep the tables (and
+    so the workspaces) alive on every rank for as long as they live, so the
+    peers' mapped pointers stay valid; pass them to ``privatized_partitioned``
+    to reuse the mappings across calls, ``close()`` them when done."""
+    jp = _engine(engine)
+    out = {}
+    for name in ("keys_A", "keys_T"):
+        t = _region(ws, loop, name, torch.int64, jp)
+        if t is not None and t.numel() <= P2P_MAX_LEN:
+            out[name] = P2PMerge(t, group)
+    return out
 
 
 def _reduce_tables(tabs, empty, group, exchange, jp):
@@ -227,11 +239,13 @@ def profile_partitioned(loop, ws, group=None, engine=None, exchange: str = "dens
     return p
 
 
-def privatized_partitioned(loop, ws, prof, group=None, engine=None, exchange: str = "dense"):
+def privatized_partitioned(loop, ws, prof, group=None, engine=None, exchange: str = "dense", p2p=None):
     """PE(V) over rank-local ranges: keys locally, C4 (MAX over packed keys), then
     every rank applies the merged keys -- each rank ends with the sequential
     result in its replica of the keyed arrays; identity-indexed outputs stay
-    sharded (each rank holds its own range)."""
+    sharded (each rank holds its own range).  ``exchange="p2p"``: small key
+    tables merge over peer memory, through ``p2p`` (from ``p2p_handles``) or
+    through handles built (collectively) and closed inside this call."""
     jp = _engine(engine)
     world, _ = world_rank(group)
     jp.jp_priv_stream(loop, prof, ws, clear_keys=True)
@@ -239,14 +253,24 @@ def privatized_partitioned(loop, ws, prof, group=None, engine=None, exchange: st
     tabs = [(name, _region(ws, loop, name, torch.int64, jp)) for name in ("keys_A", "keys_T")]
     tabs = [(n_, t) for n_, t in tabs if t is not None]
     if world > 1:
-        for name, t in tabs:
-            if exchange == "p2p" and t.numel() <= P2P_MAX_LEN:
-                arr = loop.tensors["A" if name == "keys_A" else "T"]
-                _p2p_for(t, group).run(arr=arr.view(torch.int32) if arr is not None else None)
-                applied += 1
-                continue
-            for t2 in _reduce_tables([t], 0, group, "owner" if exchange == "owner" else "dense", jp):
-                owner_reduce_replicate(t2, 0, group, jp)
+        own = None
+        if exchange == "p2p" and p2p is None and any(t.numel() <= P2P_MAX_LEN for _, t in tabs):
+            p2p = own = p2p_handles(loop, ws, group, jp)
+        try:
+            for name, t in tabs:
+                if exchange == "p2p" and t.numel() <= P2P_MAX_LEN:
+                    arr = loop.tensors["A" if name == "keys_A" else "T"]
+                    p2p[name].run(t, arr=arr.view(torch.int32) if arr is not None else None)
+                    applied += 1
+                    continue
+                for t2 in _reduce_tables([t], 0, group, "owner" if exchange == "owner" else "dense", jp):
+                    owner_reduce_replicate(t2, 0, group, jp)
+        finally:
+            if own is not None:
+                torch.cuda.synchronize()
+                dist.barrier(group=group)   # no peer still reads a table before it is unmapped
+                for h in own.values():
+                    h.close()
     if applied < len(tabs) or not tabs:
         jp.jp_priv_finalize(loop, ws)
 

@@ -222,11 +222,15 @@ def test_bad_arguments():
 
 @pytest.mark.parametrize("n,raw", [(1 << 24, 16777), (1 << 24, 167772), (1 << 24, 1677722), (4096, 205), (100, 0),
                                    (100, -1), (1000, 3), (7, 7), (1 << 20, 1)])
-def test_tls_first_window_matches_oracle(n, raw):
-    """The binding's host copy of reading A8's first window (used to label the
-    bench path) equals the oracle's definition."""
+def test_tls_next_window_matches_oracle(n, raw):
+    """The library's reading-A8 policy (the C function every TLS kernel uses)
+    equals the oracle's, for the first window and for every step."""
     for w_max in (32, 4096, 65536):
-        assert jp.tls_first_window(n, raw, w_max) == O.tls_next_window(n, raw, -1, w_max)
+        assert jp.jp_tls_next_window(n, raw, -1, w_max) == O.tls_next_window(n, raw, -1, w_max)
+        for prev in (0, 1, 15, 16, 17, 100, 4095, 4096, 70000):
+            assert jp.jp_tls_next_window(n, raw, prev, w_max) == O.tls_next_window(n, raw, prev, w_max)
+    assert jp.jp_tls_next_window(-1, raw, -1, 4096) == -1
+    assert jp.jp_tls_next_window(n, raw, -1, 16) == -1
 
 
 @pytest.mark.parametrize("seed", range(12))

@@ -1034,3 +1034,24 @@ def test_priv_tmp_slot_count_profile(seed, n, slots, full, monkeypatch):
     Ls = jp.Loop.from_workload(gpu(sub))
     ps = jp.jp_profile_density(Ls, jp.workspace(Ls))
     assert (ps["war_iters"], ps["waw_iters"]) == (rs["war_iters"], rs["waw_iters"])
+    # ranges with iter_base > 0 whose first writers lie partly OUTSIDE the range:
+    # stamp [0, b) and [b, n) into their own workspaces, MAX-combine the T tables
+    # (the C1 all-reduce of profile_partitioned), classify each range; the sum is
+    # the whole loop's profile
+    Lw = jp.Loop.from_workload(gw)
+    parts = [Lw.range(0, b), Lw.range(b, n)]
+    wss = [jp.workspace(P) for P in parts]
+    for P, W_ in zip(parts, wss):
+        jp.jp_profile_stamp(P, W_)
+    for name in ("minW_T", "minR_T"):
+        offs = [jp.jp_ws_region(P, name) for P in parts]
+        if offs[0][1] == 0:
+            continue
+        views = [W_[o:o + nb].view(torch.int32) for W_, (o, nb) in zip(wss, offs)]
+        m = torch.maximum(views[0], views[1])
+        for v in views:
+            v.copy_(m)
+    got = [jp.jp_profile_classify(P, W_) for P, W_ in zip(parts, wss)]
+    assert sum(q["raw_iters"] for q in got) == 0
+    assert sum(q["war_iters"] for q in got) == ref["war_iters"]
+    assert sum(q["waw_iters"] for q in got) == ref["waw_iters"]
