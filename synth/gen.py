@@ -246,3 +246,23 @@ def workflow_crypt(n: int = 1 << 24, parts: int = 8, device="cpu"):
             b, e = k * m, (n if k == parts - 1 else (k + 1) * m)
             loops.append(Workload("crypt", 1, 0, e - b, Y[b:e], r=perm[b:e], X=X, c0=C0_I32))
     return loops, [p, c, d, pi, pi2]
+
+
+# IEEE binary32 specials (reading A12 / A12b tests): +-0, +-inf, quiet NaNs with
+# payloads, subnormals, the normal/subnormal boundary and values near overflow
+F32_SPECIAL_BITS = [0x00000000, 0x80000000, 0x7F800000, 0xFF800000, 0x7FC00000, 0x7FC12345, 0xFFC00001,
+                    0x00000001, 0x80000001, 0x007FFFFF, 0x00800000, 0x80400000, 0x7F7FFFFF, 0xFF7FFFFF,
+                    0x7F000000, 0x00200000, 0x3F800000, 0xBF800000]
+
+
+def f32_specials(seed: int, stream: int, n: int, frac: float = 0.25, device="cpu") -> torch.Tensor:
+    """fp32 data of which about `frac` are drawn from F32_SPECIAL_BITS (chosen by
+    the counter generator) and the rest from f32_data's grid."""
+    out = f32_data(seed, stream, n, device)
+    u = rnd(seed, stream + 32, _ar(n, device))
+    pick = (_lsr(u, 11) % 1024) < int(frac * 1024)
+    which = (u & 0x3FF) % len(F32_SPECIAL_BITS)
+    table = torch.tensor(F32_SPECIAL_BITS, dtype=torch.int64, device=device)
+    bits = out.view(torch.int32).to(torch.int64) & 0xFFFFFFFF
+    bits = torch.where(pick, table[which], bits)
+    return (bits - ((bits >> 31) << 32)).to(torch.int32).view(torch.float32)
