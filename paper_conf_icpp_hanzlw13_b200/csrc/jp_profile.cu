@@ -662,6 +662,9 @@ static void run_classify(const DLoop &d, Tabs t, uint32_t *bits, int64_t chunk, 
       } else if (bits) {
         k_prof_count4<OP, true><<<grid_resident((const void *)k_prof_count4<OP, true>, g, 256, 0), 256, 0, st>>>(
             d, t, idx_vec(d), hdr, bits, src_bits, chunk, cc);
+      } else if (t.pA) {   // stamped as pairs (no guide: restart recovery asked for)
+        k_prof_count4<OP, false, true><<<grid_resident((const void *)k_prof_count4<OP, false, true>, g, 256, 0), 256,
+                                         0, st>>>(d, t, idx_vec(d), hdr, nullptr, nullptr, chunk, cc);
       } else {
         k_prof_count4<OP, false><<<grid_resident((const void *)k_prof_count4<OP, false>, g, 256, 0), 256, 0, st>>>(
             d, t, idx_vec(d), hdr, nullptr, nullptr, chunk, cc);

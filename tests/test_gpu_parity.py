@@ -556,7 +556,7 @@ def test_schedule_modes_fig2b():
         check_arrays(g, A, T)
 
 
-@pytest.mark.parametrize("n,chunk", [(1 << 16, 1024), ((1 << 18), 4096)])
+@pytest.mark.parametrize("n,chunk", [(1 << 16, 1024), ((1 << 18), 4096), ((1 << 20), 1 << 16)])
 @pytest.mark.parametrize("recovery", [0, 1])
 def test_schedule_stealing_config5(n, chunk, recovery):
     """recovery 0 (auto): the write-once TLS task runs with on-chip recovery on a
