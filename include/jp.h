@@ -148,14 +148,19 @@ typedef struct {
                                    2 on-chip.  With tls_path 0 and tls_recovery 0
                                    a SEQ_RECOMMENDED loop (mode C) runs on the
                                    one-warp program-order path 7              */
-  int32_t static_check;         /* 0: jp_static_check before profiling (affine,
-                                   conflict-free loops run as DOALL unprofiled);
-                                   1: skip it                                     */
+  int32_t static_check;         /* 0: before profiling, (a) structural RAW-freedom
+                                   (reading B11: PRIV_TMP, and SAXPY with identity
+                                   writes, cannot have a true dependence: run
+                                   privatized / DOALL after a device check of the
+                                   indirect indices, no profile), then (b)
+                                   jp_static_check (affine, conflict-free loops
+                                   run as DOALL unprofiled); 1: always profile */
 } jp_sched_cfg;
 
 typedef struct {
   int32_t mode;                 /* jp_mode of the loop (STEALING: of the first task)  */
-  int32_t profiled;             /* 0 when decided statically (all indices NULL)       */
+  int32_t profiled;             /* 0 when decided statically (all indices NULL,
+                                   affine and conflict-free, or reading B11)   */
   jp_profile prof;
   jp_tls_stats tls;
   int64_t n_tasks;              /* STEALING: same-mode chunk runs                     */

@@ -1401,6 +1401,17 @@ jp_status jp_export_keys(const jp_loop *L, void *ws, size_t ws_bytes, jp_stream_
   return JP_OK;
 }
 
+// Reading B11: the mode a loop's access sets fix without looking at its indices,
+// -1 when the indices decide.  PRIV_TMP reads only X (never written; T's read is
+// covered by the same iteration's write): RAW-free, with WAR / WAW through s or w
+// possible -> privatized (DOALL when neither is indirect).  SAXPY with identity
+// writes: Y[i] is read and written by iteration i alone, X is read-only -> DOALL.
+static int structural_mode(const Job &j) {
+  if (j.op == JP_OP_PRIV_TMP) return (j.d.s || j.d.w) ? JP_MODE_PRIVATIZED : JP_MODE_DOALL;
+  if (j.op == JP_OP_SAXPY && !j.d.w) return JP_MODE_DOALL;
+  return -1;
+}
+
 jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size_t ws_bytes, jp_sched_result *res,
                       jp_stream_t stp) {
   JP_TRY(check_loop(L));
@@ -1469,6 +1480,40 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
       res->tls_cluster = 1;
     }
     return JP_OK;
+  }
+  // structural RAW-freedom (reading B11; the paper's static rule 3, P:L257-260,
+  // "all pairs comprising a live-out and a live-in variable"): when no exposed
+  // read can touch an array that some iteration writes, d_raw = 0 whatever the
+  // indices hold, so Fig. 2(b) can only end in D or D'.  Privatized execution is
+  // exact in both, DOALL in D' -- no profile: the indirect index arrays are
+  // validated on the device and the run, launched behind it, exits at once on
+  // an out-of-range index (nothing modified, reading A13).
+  if (c.static_check == 0 && c.tls_path == 0 && ws) {
+    const int smode = structural_mode(j);
+    if (smode >= 0) {
+      Layout lo;
+      JP_TRY(check_ws(L, ws, ws_bytes, smode == JP_MODE_PRIVATIZED ? JP_WS_PRIV : 0, lo));
+      int64_t *bad = &at<int64_t>(ws, lo, R_HEADER)[H_BAD];
+      JP_CUDA(launch_validate_indirect(j, bad, st), "validate");
+      Job jr = j;
+      jr.d.abort = bad;
+      if (smode == JP_MODE_PRIVATIZED) {
+        bool applied = false;
+        JP_CUDA(launch_priv_stream(jr, ws, lo, true, st, 0, true, &applied), "priv stream");
+        if (!applied) JP_CUDA(launch_priv_finalize(jr, ws, lo, st), "priv finalize");
+      } else {
+        JP_CUDA(launch_doall(jr, st), "doall");
+      }
+      int64_t nb = 0;
+      JP_CUDA(d2h_small_sync(&nb, bad, sizeof nb, st), "validate D2H");
+      if (nb) return fail(JP_ERR_INDEX, "%lld index entries are outside their arrays", (long long)nb);
+      res->mode = smode;
+      res->profiled = 0;
+      res->n_tasks = 1;
+      res->n_batches = 1;
+      res->task_mode_iters[smode] = L->n;
+      return JP_OK;
+    }
   }
   // the pair table of the profile (all ones = no stamp yet) is filled on a side
   // stream from the start, overlapping the static check's prefix read

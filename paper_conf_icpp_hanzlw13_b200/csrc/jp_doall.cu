@@ -152,6 +152,7 @@ __global__ void __launch_bounds__(kTmaThreads, 1) k_doall_affine_tma(DLoop L, in
 
 template <int OP, int DT>
 __global__ void __launch_bounds__(256) k_doall_generic(DLoop L) {
+  if (aborted(L)) return;
   const int64_t stride = (int64_t)gridDim.x * blockDim.x;
   for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < L.n; i += stride) {
     uint32_t va = 0, vt = 0;
@@ -183,6 +184,7 @@ __device__ __forceinline__ int q_get(const int4 &v, int k) { return k == 0 ? v.x
 
 template <int OP, int DT>
 __global__ void __launch_bounds__(256) k_doall_quad(DLoop L, int vec) {
+  if (aborted(L)) return;
   constexpr int Q = 2;   // quads per thread per trip
   const int64_t nq = (L.n + 3) >> 2, B = blockDim.x;
   for (int64_t q0 = (int64_t)blockIdx.x * B * Q + threadIdx.x; q0 < nq; q0 += (int64_t)gridDim.x * B * Q) {

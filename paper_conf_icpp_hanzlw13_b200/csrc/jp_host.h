@@ -44,6 +44,9 @@ Job make_job(const jp_loop *L);
 
 // ---- launchers (each returns the first CUDA error, if any) ----
 cudaError_t launch_validate(const Job &j, int64_t *hdr, cudaStream_t st);
+// the index arrays reached through an index (identity accesses are checked on the
+// host by check_loop) against their lengths: *bad = number out of range; no sync
+cudaError_t launch_validate_indirect(const Job &j, int64_t *bad, cudaStream_t st);
 // TLS guide bitmaps (region R_GUIDE: raw words then source words) from the
 // stamp tables of a profile on the same workspace; no sync.
 cudaError_t launch_tls_guide(const Job &j, void *ws, const Layout &lo, cudaStream_t st);

@@ -54,7 +54,15 @@ struct DLoop {
   const uint32_t *X; int64_t lenX;
   uint32_t *T; int64_t lenT;
   uint32_t c0, c1;
+  // nullable device flag (the index-validation count): kernels of a run that
+  // was launched before its validation result is known exit at once when it is
+  // nonzero, so an out-of-range index still leaves every array untouched (A13)
+  const int64_t *abort = nullptr;
 };
+
+__device__ __forceinline__ bool aborted(const DLoop &L) {
+  return L.abort && *reinterpret_cast<const volatile int64_t *>(L.abort) != 0;
+}
 
 // index of local iteration i through index array p (NULL => identity)
 __host__ __device__ inline int64_t ixl(const DLoop &L, const int32_t *p, int64_t i) {

@@ -35,6 +35,7 @@ __device__ __forceinline__ void smem_last(uint32_t *tab, int64_t a, int64_t i) {
 template <int OP, int DT>
 __global__ void __launch_bounds__(kPrivThreads) k_priv_generic(DLoop L, unsigned long long *kA,
                                                                 unsigned long long *kT, int smA, int smT) {
+  if (aborted(L)) return;
   extern __shared__ uint32_t sm[];
   uint32_t *tA = smA ? sm : nullptr;
   uint32_t *tT = smT ? sm + (smA ? L.lenA : 0) : nullptr;
@@ -90,6 +91,7 @@ __global__ void __launch_bounds__(kPrivThreads) k_priv_generic(DLoop L, unsigned
 // Per iteration: X 4 B + s 4 B read, Y 4 B written (12 B/iter algorithmic).
 template <int DT>
 __global__ void __launch_bounds__(kPrivThreads) k_priv_tmp_vec(DLoop L, unsigned long long *kT, int64_t nvec) {
+  if (aborted(L)) return;
   extern __shared__ uint32_t tT[];
   for (int64_t k = threadIdx.x; k < L.lenT; k += blockDim.x) tT[k] = 0;
   JP_CTA_SYNC();
@@ -156,6 +158,7 @@ constexpr int kPrivTile = 4096, kPrivStages = 4, kPrivTmaThreads = 256;
 template <int DT>
 __global__ void __launch_bounds__(kPrivTmaThreads, 1) k_priv_tmp_tma(DLoop L, unsigned long long *kT, int64_t ntiles,
                                                                      int fuse_apply) {
+  if (aborted(L)) return;
   extern __shared__ __align__(128) uint32_t psm[];   // [stage][2][tile] then tT[lenT]
   __shared__ __align__(8) unsigned long long full[kPrivStages];
   uint32_t *tT = psm + (size_t)kPrivStages * 2 * kPrivTile;
@@ -235,7 +238,8 @@ __global__ void __launch_bounds__(kPrivTmaThreads, 1) k_priv_tmp_tma(DLoop L, un
   }
 }
 
-__global__ void k_apply_keys(uint32_t *arr, int64_t len, const unsigned long long *keys) {
+__global__ void k_apply_keys(uint32_t *arr, int64_t len, const unsigned long long *keys, const int64_t *abort) {
+  if (abort && *reinterpret_cast<const volatile int64_t *>(abort)) return;
   const int64_t stride = (int64_t)gridDim.x * blockDim.x;
   for (int64_t a = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; a < len; a += stride) {
     const unsigned long long k = keys[a];
@@ -314,16 +318,17 @@ cudaError_t launch_priv_stream(const Job &j, void *ws, const Layout &lo, bool cl
   return launch_check();
 }
 
-static void apply(uint32_t *arr, int64_t len, const unsigned long long *keys, cudaStream_t st) {
+static void apply(uint32_t *arr, int64_t len, const unsigned long long *keys, cudaStream_t st,
+                  const int64_t *abort = nullptr) {
   if (!len || !keys) return;
   int64_t need = (len + 255) / 256, cap = (int64_t)num_sms() * 8;
-  k_apply_keys<<<(int)(need < cap ? need : cap), 256, 0, st>>>(arr, len, keys);
+  k_apply_keys<<<(int)(need < cap ? need : cap), 256, 0, st>>>(arr, len, keys, abort);
   note_launch();
 }
 
 cudaError_t launch_priv_finalize(const Job &j, void *ws, const Layout &lo, cudaStream_t st) {
-  apply(j.d.A, j.d.lenA, at<unsigned long long>(ws, lo, R_KEYS_A), st);
-  if (j.op == JP_OP_PRIV_TMP) apply(j.d.T, j.d.lenT, at<unsigned long long>(ws, lo, R_KEYS_T), st);
+  apply(j.d.A, j.d.lenA, at<unsigned long long>(ws, lo, R_KEYS_A), st, j.d.abort);
+  if (j.op == JP_OP_PRIV_TMP) apply(j.d.T, j.d.lenT, at<unsigned long long>(ws, lo, R_KEYS_T), st, j.d.abort);
   return launch_check();
 }
 

@@ -531,6 +531,32 @@ __global__ void __launch_bounds__(256) k_validate(DLoop L, int64_t *hdr) {
   if ((threadIdx.x & 31) == 0 && bad) atomicAdd((unsigned long long *)&hdr[H_BAD], (unsigned long long)bad);
 }
 
+// one index array against its length: 16-byte loads, four in flight per thread
+// (a stream at HBM rate; the structural path's only pass before the run)
+__global__ void __launch_bounds__(256) k_check_idx(const int32_t *p, int64_t n, int64_t len, int64_t *bad_out) {
+  int64_t bad = 0;
+  const int64_t stride = (int64_t)gridDim.x * blockDim.x, tid = (int64_t)blockIdx.x * blockDim.x + threadIdx.x;
+  const int64_t head = ((uintptr_t)p & 15) ? (16 - ((uintptr_t)p & 15)) / 4 : 0;
+  const int64_t h = head < n ? head : n;
+  if (tid < h) bad += (uint32_t)p[tid] >= (uint64_t)len;
+  const int4 *p4 = reinterpret_cast<const int4 *>(p + h);
+  const int64_t nv = (n - h) >> 2;
+  auto chk = [&](int4 v) {
+    bad += ((uint32_t)v.x >= (uint64_t)len) + ((uint32_t)v.y >= (uint64_t)len) + ((uint32_t)v.z >= (uint64_t)len) +
+           ((uint32_t)v.w >= (uint64_t)len);
+  };
+  int64_t v = tid;
+  for (; v + 3 * stride < nv; v += 4 * stride) {
+    const int4 a = __ldcs(p4 + v), b = __ldcs(p4 + v + stride), c = __ldcs(p4 + v + 2 * stride),
+               d = __ldcs(p4 + v + 3 * stride);
+    chk(a); chk(b); chk(c); chk(d);
+  }
+  for (; v < nv; v += stride) chk(__ldcs(p4 + v));
+  for (int64_t i = h + 4 * nv + tid; i < n; i += stride) bad += (uint32_t)p[i] >= (uint64_t)len;
+  for (int o = 16; o; o >>= 1) bad += __shfl_xor_sync(0xffffffffu, bad, o);
+  if ((threadIdx.x & 31) == 0 && bad) atomicAdd((unsigned long long *)bad_out, (unsigned long long)bad);
+}
+
 static int grid_for(int64_t n, int threads, int per_sm) {
   int64_t need = (n + threads - 1) / threads;
   int64_t cap = (int64_t)num_sms() * per_sm;
@@ -831,6 +857,23 @@ cudaError_t launch_tls_guide(const Job &j, void *ws, const Layout &lo, cudaStrea
   if (!bits || !maxRx || !minW || j.d.n == 0) return launch_check();
   cudaMemsetAsync(maxRx, 0xFF, lo.bytes[R_MAXRX_A], st);
   JP_DISPATCH(j.op, j.dt, run_guide, j.d, minW, maxRx, bits, st);
+  return launch_check();
+}
+
+cudaError_t launch_validate_indirect(const Job &j, int64_t *bad, cudaStream_t st) {
+  cudaMemsetAsync(bad, 0, sizeof(int64_t), st);
+  const DLoop &d = j.d;
+  auto one = [&](const int32_t *p, int64_t len) {
+    if (!p || d.n == 0) return;
+    k_check_idx<<<grid_for((d.n + 3) / 4, 256, 8), 256, 0, st>>>(p, d.n, len, bad);
+    note_launch();
+  };
+  switch (j.op) {
+    case JP_OP_ADD_C: one(d.r, d.lenA); one(d.w, d.lenA); break;
+    case JP_OP_SAXPY: one(d.r, d.lenX); one(d.w, d.lenA); break;
+    case JP_OP_PRIV_TMP: one(d.r, d.lenX); one(d.s, d.lenT); one(d.w, d.lenA); break;
+    default: one(d.r, d.lenA); one(d.r2, d.lenA); one(d.w, d.lenA);
+  }
   return launch_check();
 }
 

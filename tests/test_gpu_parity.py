@@ -160,6 +160,50 @@ def test_index_error_no_side_effects():
     assert jp.jp_validate(L, ws) == 1
 
 
+@pytest.mark.parametrize("case", ["c4", "c4_w", "saxpy_r"])
+def test_structural_raw_free_schedule(case):
+    """Reading B11: PRIV_TMP (X read-only, T's read covered) and SAXPY with
+    identity writes are run without a profile (profiled = 0) -- results equal the
+    oracle; an out-of-range indirect index gives JP_ERR_INDEX with every array
+    untouched (the run launched behind the device check exits at once)."""
+    n = (1 << 20) + 77
+    g0 = np.random.default_rng(3)
+    if case == "c4":
+        wl, mode = synth.config4(n=n), jp.JP_MODE_PRIVATIZED
+    elif case == "c4_w":   # Y written through a 2-to-1 index: WAW on Y as well
+        wl, mode = synth.config4(n=n), jp.JP_MODE_PRIVATIZED
+        wl.w = torch.from_numpy((g0.permutation(n) // 2).astype(np.int32))
+    else:
+        wl, mode = random_loop(9, O.OP_SAXPY, O.F32, n, null_prob=0.0), jp.JP_MODE_DOALL
+        wl.w = None
+    _, A, T = O.run_seq(to_oracle(wl))
+    g = gpu(wl)
+    L = jp.Loop.from_workload(g)
+    ws = jp.workspace(L)
+    res = jp.jp_schedule(L, ws)
+    torch.cuda.synchronize()
+    assert res["mode"] == mode and res["profiled"] == 0, res
+    check_arrays(g, A, T)
+    # the same loop with one bad indirect index: nothing modified
+    g = gpu(wl)
+    idx = g.s if case.startswith("c4") else g.r
+    idx[n // 2] = 1 << 30
+    A0, T0 = g.A.clone(), None if g.T is None else g.T.clone()
+    L = jp.Loop.from_workload(g)
+    with pytest.raises(jp.JPError) as e:
+        jp.jp_schedule(L, ws)
+    assert e.value.status == -5
+    torch.cuda.synchronize()
+    assert torch.equal(g.A, A0) and (T0 is None or torch.equal(g.T, T0))
+    # static_check = 1: the profile decides (Fig. 2(b)), same arrays
+    g = gpu(wl)
+    L = jp.Loop.from_workload(g)
+    res = jp.jp_schedule(L, ws, static_check=1)
+    torch.cuda.synchronize()
+    assert res["profiled"] == 1 and res["prof"]["raw_iters"] == 0
+    check_arrays(g, A, T)
+
+
 def test_illegal_modes_and_workspace():
     wl = synth.config1(0.05)
     g = gpu(wl)
@@ -234,7 +278,10 @@ def test_doall_indirect_permutation(op, dt):
     g = gpu(wl)
     L = jp.Loop.from_workload(g)
     res = jp.jp_schedule(L, jp.workspace(L))
-    assert res["mode"] == jp.JP_MODE_DOALL and res["profiled"] == 1
+    if op == O.OP_PRIV_TMP:   # reading B11: RAW-free by its access sets, privatized without a profile
+        assert res["mode"] == jp.JP_MODE_PRIVATIZED and res["profiled"] == 0
+    else:
+        assert res["mode"] == jp.JP_MODE_DOALL and res["profiled"] == 1
     torch.cuda.synchronize()
     check_arrays(g, A, T)
 
@@ -818,7 +865,7 @@ def test_schedule_profile_interleaved_tables(op, seed, pairs, monkeypatch):
     p = O.profile(ref)
     g = gpu(wl)
     L = jp.Loop.from_workload(g)
-    res = jp.jp_schedule(L, jp.workspace(L), tls_recovery=1)
+    res = jp.jp_schedule(L, jp.workspace(L), tls_recovery=1, static_check=1)
     torch.cuda.synchronize()
     assert (res["prof"]["raw_iters"], res["prof"]["war_iters"], res["prof"]["waw_iters"],
             res["prof"]["first_raw_iter"]) == (p["raw_iters"], p["war_iters"], p["waw_iters"], p["first_raw_iter"])

@@ -104,7 +104,7 @@ def test_specials_doall_indirect(op, generic, monkeypatch):
     _, A, T = O.run_seq(to_oracle(wl))
     g = wl.to(DEV)
     L = jp.Loop.from_workload(g)
-    res = jp.jp_schedule(L, jp.workspace(L))
+    res = jp.jp_schedule(L, jp.workspace(L), static_check=1)
     torch.cuda.synchronize()
     assert res["mode"] == jp.JP_MODE_DOALL
     check(g, A, T)
