@@ -160,6 +160,28 @@ def config3(density: float = 0.01, n: int = 1 << 24, delta: int = 1024, device="
                     meta={"raw": k, "war": 0, "waw": 0, "delta": delta, "density": density})
 
 
+def config3_waw(density: float = 0.01, n: int = 1 << 24, delta: int = 1024, device="cpu") -> Workload:
+    """Config 3's shape with write-after-write (the loop on which on-chip
+    recovery, reading B7, is illegal and restart TLS must run): w is 2-to-1
+    onto [0, n/2) (w[i] = pi[i] >> 1); an independent iteration reads the
+    read-only half [n/2, n) (n/2 + (pi2[i] >> 1)); the K = round(d*n) dependent
+    iterations (same choice as config 3) read w[i - delta_i].  Designed
+    profile: raw = K, waw = n/2 exactly."""
+    assert n % 2 == 0
+    seed = 1013
+    w = _lsr(permutation(seed, n, device), 1)
+    r = n // 2 + _lsr(permutation(seed + 1, n, device), 1)
+    k = int(round(density * n))
+    dep = dependent_set(seed, n, k, device)
+    if k:
+        m = torch.clamp(dep, max=delta)
+        d = 1 + _lsr(rnd(seed, 5, dep), 1) % m
+        r[dep] = w[dep - d]
+    return Workload("config3_waw", 0, 0, n, i32_data(seed, 1, n, device), r=r.to(torch.int32),
+                    w=w.to(torch.int32), c0=C0_I32, meta={"raw": k, "waw": n // 2, "delta": delta,
+                                                          "density": density})
+
+
 def config4(n: int = 1 << 26, slots: int = 1024, device="cpu") -> Workload:
     """Config 4: PRIV_TMP fp32, s[i] = rnd(seed,3,i) mod S (S = 1024 scratch slots)."""
     seed = 1004

@@ -1,5 +1,6 @@
 """Generator tests: counter-based draws, determinism, and designed densities."""
 import numpy as np
+import pytest
 import torch
 
 import oracle as O
@@ -94,3 +95,15 @@ def test_device_agnostic_bits():
     b = synth.config4(n=4096)
     for k in ("s", "X", "T", "A"):
         assert torch.equal(getattr(a, k), getattr(b, k))
+
+
+@pytest.mark.parametrize("d,delta", [(0.0, 1024), (0.01, 1024), (0.1, 64), (0.05, 1 << 20)])
+def test_config3_waw_designed_profile(d, delta):
+    """The WAW variant of config 3: raw = K exactly, waw = n/2 exactly (every
+    address of [0, n/2) written twice), against the oracle's profile."""
+    n = 1 << 13
+    wl = synth.config3_waw(d, n=n, delta=delta)
+    p = O.profile(_oracle_loop(wl))
+    assert (p["raw_iters"], p["waw_iters"]) == (wl.meta["raw"], n // 2)
+    assert wl.meta["raw"] == round(d * n)
+    assert int(wl.w.max()) < n // 2 and int(wl.r.max()) < n
