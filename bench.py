@@ -156,15 +156,35 @@ def oracle_baseline(sample_iters: int, max_runs: int = 5, budget_s: float = 10.0
     box's host on a bounded sample of the same workload."""
     O, L = oracle_loop(sample_iters)
     O.run_seq_inplace(L)  # warm (and build) the .so
-    times, t_end = [], time.perf_counter() + budget_s
-    while not times or (len(times) < max_runs and time.perf_counter() < t_end):
-        t0 = time.perf_counter()
-        O.run_seq_inplace(L)
-        times.append(time.perf_counter() - t0)
+    old = os.sched_getaffinity(0)
+    cpu = min(old)
+    os.sched_setaffinity(0, {cpu})   # one core, as `taskset -c 0` (SURVEY Sec.8(d))
+    try:
+        times, t_end = [], time.perf_counter() + budget_s
+        while not times or (len(times) < max_runs and time.perf_counter() < t_end):
+            t0 = time.perf_counter()
+            O.run_seq_inplace(L)
+            times.append(time.perf_counter() - t0)
+    finally:
+        os.sched_setaffinity(0, old)
     t = statistics.median(times)
     return {"value": sample_iters / t, "unit": "iter/s", "cores": 1, "kind": "oracle", "cpu_model": _cpu_model(),
+            "pinned_cpu": cpu,
             "sample": f"config2 SAXPY fp32, first {sample_iters} of the 2^28 iterations, jpo_run_seq on 1 host "
-                      f"thread of {os.cpu_count()}, median of {len(times)} runs ({t:.3f} s each)"}
+                      f"thread (pinned to cpu {cpu}) of {os.cpu_count()}, median of {len(times)} runs "
+                      f"({t:.3f} s each)"}
+
+
+# The paper's own numbers are context, not the target (BASELINE.md): another
+# machine, another workload mix, a different program (Java + JNI + Fermi).
+PAPER_CONTEXT = {
+    "source": "Han, Zhang, Lam, Wang, ICPP'13 (PAPER.md L41-43 abstract; L471-491 Sec. VI setup)",
+    "platform": "NVIDIA Tesla M2050 (Fermi, CUDA 3.2) + 2x Intel Xeon X5650 (12 cores), Java 1.6",
+    "speedups_vs_serial_cpu": {"doall_loops": "10x (average)", "false_dependence_privatized": "2.5x",
+                               "true_dependence_density_low": "2.14x"},
+    "note": "speedups of whole Java applications over a 1-thread CPU run, on Fermi; the bench here reports "
+            "committed iterations/s and HBM fraction of the loop hot path on one B200, with the CPU oracle "
+            "(1 core) beside it"}
 
 
 def _cpu_model() -> str:
@@ -195,11 +215,14 @@ def run_reference(args):
     sample = 1 << 25
     O, L = oracle_loop(sample)
     times = []
+    old = os.sched_getaffinity(0)
+    os.sched_setaffinity(0, {min(old)})   # one host core (taskset -c 0)
     for k in range(args.warmup + args.steps):
         t0 = time.perf_counter()
         O.run_seq_inplace(L)
         if k >= args.warmup:
             times.append(time.perf_counter() - t0)
+    os.sched_setaffinity(0, old)
     t = statistics.mean(times)
     v = sample / t
     print(json.dumps({"impl": "reference", "metric": METRIC, "value": v, "unit": "iter/s", "n_gpus": args.gpus,
@@ -226,6 +249,91 @@ def time_steps(fn, steps, st):
     return [a.elapsed_time(b) for a, b in ev]
 
 
+def median_timed(fn, A, A0, st, reps=None, budget_ms=2500.0):
+    out, ts = None, []
+    for k in range(3):   # warm-up
+        if A is not None:
+            A.copy_(A0)
+        torch.cuda.synchronize()
+        a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        a.record(st)
+        out = fn()
+        b.record(st)
+        torch.cuda.synchronize()
+        if k == 0 and a.elapsed_time(b) > 300:   # slow call: one warm-up is enough
+            break
+    first = a.elapsed_time(b)
+    k = reps if reps is not None else int(min(20, max(3, budget_ms / max(first, 1e-3))))
+    for _ in range(k):
+        if A is not None:
+            A.copy_(A0)
+        torch.cuda.synchronize()
+        a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        a.record(st)
+        out = fn()
+        b.record(st)
+        torch.cuda.synchronize()
+        ts.append(a.elapsed_time(b))
+    return out, statistics.median(ts)
+
+
+def pinned_oracle_rate(loop, budget_s: float = 1.0) -> float:
+    """The CPU oracle (jpo_run_seq) on one host core (the calling thread pinned
+    to the first allowed CPU, as `taskset -c 0` would), iterations per second:
+    median of up to 5 runs within the budget."""
+    import oracle as O
+    old = os.sched_getaffinity(0)
+    os.sched_setaffinity(0, {min(old)})
+    try:
+        ts, t_end = [], time.perf_counter() + budget_s
+        while not ts or (len(ts) < 5 and time.perf_counter() < t_end):
+            L = loop.copy()
+            t0 = time.perf_counter()
+            O.run_seq_inplace(L)
+            ts.append(time.perf_counter() - t0)
+    finally:
+        os.sched_setaffinity(0, old)
+    return loop.n / statistics.median(ts)
+
+
+def crossover_sweep(jp, dev, st, n=1 << 20):
+    """Reading A4's tau_high, measured (Fig. 2(b) "(Density > N)", P:L399-410;
+    mode C P:L375-378): committed iter/s of the whole jp_schedule call with
+    on-chip TLS (B7), restart TLS (A6) and the one-warp program-order path 7,
+    against the 1-thread CPU oracle, over true-RAW densities 10-100%, for the
+    config-3 recipe (delta <= 1024) and for chains (delta = 1: r[i] = w[i-1])."""
+    import oracle as O
+    import synth
+    rows = []
+    for delta in (1024, 1):
+        for d in (0.10, 0.25, 0.50, 0.75, 1.0):
+            wl = synth.config3(d, n=n, delta=delta, device=dev)
+            ref = O.Loop(wl.op, wl.dtype, wl.n, wl.A.cpu().numpy(), r=wl.r.cpu().numpy(), w=wl.w.cpu().numpy(),
+                         c0=wl.c0)
+            A0 = wl.A.clone()
+            L = jp.Loop.from_workload(wl)
+            ws = jp.workspace(L)
+            row = {"delta": delta, "density": d}
+            for name, kw in (("onchip", dict(tau_high=1.0, tls_recovery=2)),
+                             ("restart", dict(tau_high=1.0, tls_recovery=1)),
+                             ("serial_path7", dict(tau_high=1e-9))):
+                res, ms = median_timed(lambda: jp.jp_schedule(L, ws, stream=st, **kw), wl.A, A0, st, budget_ms=1500)
+                row[name] = n / (ms * 1e-3)
+                row["raw_iters"] = res["prof"]["raw_iters"]
+            row["oracle_1core"] = pinned_oracle_rate(ref)
+            rows.append(row)
+            del wl, ws, L, A0, ref
+    out = {"rows": rows, "n": n, "unit": "committed iter/s, whole jp_schedule call, median"}
+    for delta in (1024, 1):
+        rs = [r for r in rows if r["delta"] == delta]
+        tls_best = lambda r: max(r["onchip"], r["restart"])  # noqa: E731
+        a = [r["density"] for r in rs if r["serial_path7"] >= tls_best(r)]
+        b = [r["density"] for r in rs if r["oracle_1core"] > max(tls_best(r), r["serial_path7"])]
+        out[f"delta{delta}"] = {"serial_beats_tls_from_density": min(a) if a else None,
+                                "cpu_beats_gpu_from_density": min(b) if b else None}
+    return out
+
+
 def modes_sweep(jp, dev, st):
     """N=1 extras: TLS vs density (config 3), privatized (config 4), tiny (config 1), mixed (config 5)."""
     import synth
@@ -240,17 +348,11 @@ def modes_sweep(jp, dev, st):
     tls = []
     names = {1: "cta", 2: "grid", 3: "cluster16", 4: "tiny", 5: "onchip-cluster", 6: "onchip-grid"}
 
-    def timed(fn, A, A0):
-        out = None
-        for rep in range(2):   # warm-up, then timed
-            A.copy_(A0)
-            torch.cuda.synchronize()
-            a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
-            a.record(st)
-            out = fn()
-            b.record(st)
-            torch.cuda.synchronize()
-        return out, a.elapsed_time(b)
+    def timed(fn, A, A0, reps=None):
+        """warm up, then the median of `reps` timed runs (20, or
+        fewer for calls slower than ~100 ms, so the sweep ends in minutes); the
+        in-place array is restored from a pristine copy outside the timed region."""
+        return median_timed(fn, A, A0, st, reps)
 
     for d in (0.001, 0.01, 0.05, 0.10):
         wl = synth.config3(d, device=dev)
@@ -296,27 +398,52 @@ def modes_sweep(jp, dev, st):
             res, ms = timed(lambda: jp.jp_schedule(L, ws, stream=st, tls_recovery=rec), wl.A, A0)
             row[tag + "schedule"] = {"mode": res["mode_name"], "ms": ms, "committed_per_s": wl.n / (ms * 1e-3),
                                      "windows": res["tls"]["windows"], "violations": res["tls"]["violations"],
-                                     "recovery": ["restart", "onchip"][res["tls_recovery"]]}
+                                     "recovery": ["restart", "onchip"][res["tls_recovery"]],
+                                     "tls_w_max": res["tls_w_max"], "tls_path": names.get(res["tls_path"], "?")}
         sens.append(row)
         del wl, ws, L, A0
     out["config3_tls_delta_2e20"] = sens
-    # config 4: privatized (profile once, then time the privatized run alone and the whole schedule)
+    # config 3's shape WITH write-after-write (synth.config3_waw: w 2-to-1 onto half
+    # the addresses): on-chip recovery (reading B7) is illegal, so jp_schedule runs
+    # restart TLS (reading A6) with the cap / path of the distance-hazard plan
+    waw = []
+    for delta in (1024, 1 << 20):
+        for d in (0.001, 0.01, 0.05, 0.10):
+            wl = synth.config3_waw(d, delta=delta, device=dev)
+            A0 = wl.A.clone()
+            L = jp.Loop.from_workload(wl)
+            ws = jp.workspace(L)
+            res, ms = timed(lambda: jp.jp_schedule(L, ws, stream=st), wl.A, A0)
+            waw.append({"density": d, "delta": delta, "mode": res["mode_name"], "ms": ms,
+                        "committed_per_s": wl.n / (ms * 1e-3), "raw_iters": res["prof"]["raw_iters"],
+                        "waw_iters": res["prof"]["waw_iters"], "windows": res["tls"]["windows"],
+                        "violations": res["tls"]["violations"], "recovery": ["restart", "onchip"][res["tls_recovery"]],
+                        "tls_w_max": res["tls_w_max"], "tls_path": names.get(res["tls_path"], "?"),
+                        "us_per_window": ms * 1e3 / max(res["tls"]["windows"], 1)})
+            del wl, ws, L, A0
+    out["config3_waw_restart"] = waw
+    out["crossover"] = crossover_sweep(jp, dev, st)
+    # config 4: privatized.  The whole jp_schedule call (what a user runs: reading
+    # B11 decides privatized without a profile, the s indices are checked on the
+    # device, then stream + merge + apply), the privatized run alone, and the
+    # profile alone (jp_profile_density: what Fig. 2(b) would have cost)
     wl = synth.config4(device=dev)
     L = jp.Loop.from_workload(wl)
     ws = jp.workspace(L)
+    res, ms_call = timed(lambda: jp.jp_schedule(L, ws, stream=st), None, None)
     prof = jp.jp_profile_density(L, ws)
-    jp.jp_run_privatized(L, prof, ws, stream=st)
-    ms = time_steps(lambda: jp.jp_run_privatized(L, prof, ws, stream=st), 10, st)
-    t = statistics.mean(ms) * 1e-3
-    a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
-    a.record(st)
-    jp.jp_profile_density(L, ws, stream=st)
-    b.record(st)
-    torch.cuda.synchronize()
-    out["config4_priv"] = {"n": wl.n, "iters_per_s": wl.n / t, "ms": t * 1e3,
-                           "hbm_gbs": BYTES_PER_ITER_PRIV * wl.n / t / 1e9,
-                           "frac": BYTES_PER_ITER_PRIV * wl.n / t / 1e9 / hbm,
-                           "profile_ms": a.elapsed_time(b)}
+    _, ms_run = timed(lambda: jp.jp_run_privatized(L, prof, ws, stream=st), None, None)
+    _, ms_prof = timed(lambda: jp.jp_profile_density(L, ws, stream=st), None, None)
+    byt = BYTES_PER_ITER_PRIV * wl.n
+    out["config4_priv"] = {"n": wl.n, "mode": res["mode_name"], "profiled": res["profiled"],
+                           "schedule_ms": ms_call, "iters_per_s": wl.n / (ms_call * 1e-3),
+                           "schedule_hbm_gbs": byt / (ms_call * 1e-3) / 1e9,
+                           "schedule_frac": byt / (ms_call * 1e-3) / 1e9 / hbm,
+                           "run_ms": ms_run, "run_frac": byt / (ms_run * 1e-3) / 1e9 / hbm,
+                           "profile_ms": ms_prof,
+                           "algorithmic_bytes": "12 B/iter (X, s read; Y written); the device index check "
+                                                "re-reads s (4 B/iter) inside the whole call",
+                           "timing": "median of up to 20, CUDA events on the stream"}
     del wl, ws, L
     # config 1: tiny loop, latency-bound (us per jp_schedule call, incl. profile + mode + run)
     c1 = {}
@@ -348,16 +475,11 @@ def modes_sweep(jp, dev, st):
     A0 = wl.A.clone()
     L = jp.Loop.from_workload(wl)
     ws = jp.workspace(L)
-    jp.jp_schedule(L, ws, stream=st, scheme=jp.JP_SCHED_STEALING, chunk_iters=65536)
-    wl.A.copy_(A0)
-    torch.cuda.synchronize()
-    t0 = time.perf_counter()
-    res = jp.jp_schedule(L, ws, stream=st, scheme=jp.JP_SCHED_STEALING, chunk_iters=65536)
-    torch.cuda.synchronize()
-    t = time.perf_counter() - t0
-    out["config5_mixed"] = {"n": wl.n, "iters_per_s": wl.n / t, "ms": t * 1e3, "n_tasks": res["n_tasks"],
+    res, ms = timed(lambda: jp.jp_schedule(L, ws, stream=st, scheme=jp.JP_SCHED_STEALING, chunk_iters=65536),
+                    wl.A, A0)
+    out["config5_mixed"] = {"n": wl.n, "iters_per_s": wl.n / (ms * 1e-3), "ms": ms, "n_tasks": res["n_tasks"],
                             "n_batches": res["n_batches"], "task_mode_iters": res["task_mode_iters"],
-                            "tls": res["tls"]}
+                            "tls": res["tls"], "timing": "median of up to 20, CUDA events on the stream"}
     del wl, ws, L, A0
     # workflows: the paper's task-stealing shapes, N = 2^24
     # iterations per original loop, every scheme; whole jp_schedule_workflow call
@@ -419,8 +541,13 @@ def partitioned_config4(jp, dev, st, world, rank, steps):
     prof_ms = timed(lambda: prof.update(jd.profile_partitioned(loop, ws)), steps)
     mode = jp.jp_select_mode(loop, prof, 0.25)
     ms = timed(lambda: jd.privatized_partitioned(loop, ws, prof), steps)
-    ms_p2p = timed(lambda: jd.privatized_partitioned(loop, ws, prof, exchange="p2p"), steps) \
-        if world > 1 and IPC_ROWS else None
+    ms_p2p = None
+    if world > 1 and IPC_ROWS:
+        handles = jd.p2p_handles(loop, ws)   # collective, once: the IPC mappings outlive the steps
+        ms_p2p = timed(lambda: jd.privatized_partitioned(loop, ws, prof, exchange="p2p", p2p=handles), steps)
+        barrier(world)
+        for h in handles.values():
+            h.close()
     hbm, _ = peaks()
     return {"workload": "config4: PRIV_TMP fp32 N=2^26 S=1024, task sharing; step = privatized stream + C4 + finalize",
             "n": wl.n, "n_per_rank": e - b, "mode": jp.MODE_NAMES[mode], "ms": ms, "iters_per_s": wl.n / (ms * 1e-3),
@@ -670,10 +797,14 @@ def run_jp(args):
     value = N2 * args.steps / (total_ms * 1e-3)
     hbm, peak_src = peaks()
     achieved = BYTES_PER_ITER_SAXPY * (s1 - s0) / (kernel_ms * 1e-3) / 1e9
+    # ncu DRAM bytes per launch of the whole 2^28 step (profiles/ncu_doall_traffic.json,
+    # one `ncu --set full` capture of this command at N = 1), scaled to this rank's
+    # share of the iterations (the kernel streams its range exactly once)
     traffic = None
     tp = os.path.join(ROOT, "profiles", "ncu_doall_traffic.json")
     if os.path.exists(tp):
-        traffic = json.load(open(tp)).get("dram_bytes_per_launch")
+        full = json.load(open(tp)).get("dram_bytes_per_launch")
+        traffic = None if full is None else full * (s1 - s0) / N2
 
     # e2e: the same step through jp_schedule_host with pinned host buffers
     e2e_steps = min(args.steps, 3)
@@ -724,9 +855,11 @@ def run_jp(args):
                                                         "k_doall_affine_tma<SAXPY,F32>"][jp.jp_doall_kernel(-1)],
                             "achieved": achieved,
                             "peak": hbm, "unit": "GB/s", "frac": achieved / hbm, "traffic": traffic,
+                            "traffic_source": "ncu dram__bytes_read.sum + dram__bytes_write.sum per launch "
+                                              "(profiles/ncu_doall_traffic.json, N=1), x this rank's share",
                             "algorithmic_bytes_per_iter": BYTES_PER_ITER_SAXPY, "peak_source": peak_src,
                             "kernel_ms": kernel_ms},
-               "clocks": clk.summary(), "e2e": e2e, "gpu_launches": launches_all}
+               "clocks": clk.summary(), "e2e": e2e, "gpu_launches": launches_all, "paper_context": PAPER_CONTEXT}
     if not args.no_modes:
         del wl, L
         torch.cuda.empty_cache()
@@ -735,7 +868,7 @@ def run_jp(args):
         spill = partitioned_spill(jp, dev, st, world, rank, 5) if world == 1 or IPC_ROWS else \
             {"skipped": "CUDA-IPC rows at N > 1 need JP_BENCH_IPC=1"}
         torch.cuda.empty_cache()
-        steal = partitioned_config5(jp, dev, st, world, rank, 3)
+        steal = partitioned_config5(jp, dev, st, world, rank, 10)
         torch.cuda.empty_cache()
         if rank == 0:
             out["partitioned"] = {"config4": part, "config2_spill": spill, "config5_stealing": steal}

@@ -649,6 +649,91 @@ static int64_t auto_w_max(const jp_profile *p) {
   return w;
 }
 
+// Restart-TLS plan from the profile's dependence distances (reading A8's cap
+// and the path; the semantics and the oracle's statistics only depend on the
+// cap, which jp_sched_result reports).  A window starting at ws ends at the
+// first iteration whose exposed read was written inside the window: an
+// iteration at offset m is raw with probability d = raw_iters / n and then
+// violates iff its distance delta <= m, so the hazard is h(m) = d F(m) with F
+// the distance CDF (dist[b] = raw reads with floor(log2 delta) = b, F linear
+// inside a bucket).  The expected commit of a window capped at W is
+// E[c_W] = sum_{k<W} prod_{m<k} (1 - h(m)); the adaptive policy keeps windows
+// near min(W, 2 E[c]), so one committed iteration costs about
+// cost(path, min(W, 2 E[c])) / E[c_W].  cost() is the measured time per window
+// of each path at fixed windows on dependence-free loops (scripts/restart_calib.py,
+// profiles/r02_restart_calib.jsonl; B200, N = 2^22), with and without the WAW
+// commit.  The (path, W) of least cost per committed iteration wins.
+namespace {
+struct CostPt { int path; int64_t w; double us, us_waw; };
+constexpr CostPt kRestartCost[] = {
+    {1, 64, 0.85, 1.01},      {1, 128, 0.88, 1.07},     {1, 256, 0.98, 1.18},     {1, 512, 1.21, 1.57},
+    {1, 1024, 2.53, 3.04},    {3, 2048, 2.79, 4.53},    {3, 4096, 3.08, 5.26},    {3, 8192, 3.72, 6.25},
+    {3, 16384, 4.80, 8.89},   {3, 32768, 7.18, 13.96},  {3, 65536, 12.05, 24.07}, {2, 262144, 22.85, 28.72}};
+}  // namespace
+
+static double restart_cost(int path, int64_t w, bool waw) {
+  // piecewise linear in W between the measured points of the same path
+  const CostPt *lo = nullptr, *hi = nullptr;
+  for (const CostPt &c : kRestartCost) {
+    if (c.path != path) continue;
+    if (c.w <= w) lo = &c;
+    if (c.w >= w && !hi) hi = &c;
+  }
+  if (!lo) lo = hi;
+  if (!hi) hi = lo;
+  const double a = waw ? lo->us_waw : lo->us, b = waw ? hi->us_waw : hi->us;
+  if (hi->w == lo->w) return a;
+  return a + (b - a) * (double)(w - lo->w) / (double)(hi->w - lo->w);
+}
+
+// expected commit length of a window of at most W iterations (see above)
+static double restart_commit(const int64_t *dist, double d, int64_t W) {
+  double tot = 0;
+  for (int b = 0; b < 32; b++) tot += (double)dist[b];
+  if (tot <= 0 || d <= 0) return (double)W;
+  double F = 0, logS = 0, ec = 0;   // F(m) at the start of bucket b, log S(m)
+  int64_t m = 0;
+  // m = 0 never violates (delta >= 1); step through the buckets [2^b, 2^(b+1))
+  ec += 1.0;
+  m = 1;
+  for (int b = 0; b < 32 && m < W; b++) {
+    const int64_t lo = (int64_t)1 << b, hi = std::min<int64_t>((int64_t)2 << b, W);
+    const double fb = (double)dist[b] / tot;      // mass of this bucket, spread over [2^b, 2^(b+1))
+    const double span = (double)((int64_t)1 << b);
+    // integrate k over [lo, hi) in up to 64 steps: S(k) = exp(logS), logS += log(1 - d F(k))
+    const int64_t steps = std::min<int64_t>(64, hi - lo);
+    const double dk = (double)(hi - lo) / (double)steps;
+    for (int64_t q = 0; q < steps; q++) {
+      const double k = (double)lo + (q + 0.5) * dk;
+      const double Fk = F + fb * (k - (double)lo + 1.0) / span;
+      const double h = std::min(0.999999, d * Fk);
+      ec += exp(logS) * dk;
+      logS += log1p(-h) * dk;
+    }
+    F += fb;
+    m = hi;
+    if (logS < -50) break;   // every later window position is unreachable
+  }
+  return ec;
+}
+
+static void restart_plan(const jp_profile *p, const int64_t *dist, int64_t n, bool waw, int64_t *w_max, int *path) {
+  const double d = p && p->n > 0 ? (double)p->raw_iters / (double)p->n : 0.0;
+  double best = 1e300;
+  for (const CostPt &c : kRestartCost) {
+    if (c.w > std::max<int64_t>(n, 64) * 2 && c.w > 64) continue;
+    const double ec = restart_commit(dist, d, c.w);
+    double weff = std::min((double)c.w, 2.0 * ec);
+    if (weff < 32) weff = 32;
+    const double t = restart_cost(c.path, (int64_t)weff, waw) / std::max(ec, 1.0);
+    if (t < best) {
+      best = t;
+      *w_max = c.w;
+      *path = c.path;
+    }
+  }
+}
+
 // auto_guide: run jp_tls_guide first when the plan benefits (cluster path
 // always, single-CTA path at d_raw <= 2%: measured) and the profile and
 // workspace allow it (jp_schedule)
@@ -1008,7 +1093,7 @@ static Job sub_job(const Job &j, int64_t s, int64_t e) {
 
 static jp_status run_mode(const jp_loop *L, const Job &j, int mode, const jp_profile *prof, const jp_sched_cfg &c,
                           void *ws, size_t ws_bytes, jp_sched_result *res, cudaStream_t st, bool guide_ready = false,
-                          int s_clean = 0) {
+                          int s_clean = 0, const int64_t *dist = nullptr) {
   Layout lo = layout(L);
   if (mode == JP_MODE_DOALL) {
     JP_CUDA(launch_doall(j, st), "doall");
@@ -1028,8 +1113,13 @@ static jp_status run_mode(const jp_loop *L, const Job &j, int mode, const jp_pro
                     : c.tls_recovery == 1 ? JP_TLS_RESTART
                     : c.tls_recovery == 2 || (c.tls_path == 0 && prof && prof->waw_iters == 0) ? JP_TLS_ONCHIP
                                                                                             : JP_TLS_RESTART;
-    const int64_t wm = c.tls_w_max > 0 ? c.tls_w_max : auto_w_max(prof);
-    jp_tls_cfg tc{c.tls_window, wm, serial ? 7 : c.tls_path, 0, 0, rec};
+    int64_t wm = c.tls_w_max > 0 ? c.tls_w_max : auto_w_max(prof);
+    int path = serial ? 7 : c.tls_path;
+    // restart recovery with the profile's dependence distances: cap and path
+    // from the distance-hazard model (restart_plan) unless the caller fixed them
+    if (!serial && rec == JP_TLS_RESTART && dist && prof && c.tls_w_max == 0 && c.tls_path == 0 && c.tls_window == 0)
+      restart_plan(prof, dist, j.d.n, prof->waw_iters > 0, &wm, &path);
+    jp_tls_cfg tc{c.tls_window, wm, path, 0, 0, rec};
     TlsPlan tp;
     JP_TRY(run_tls_job(L, j, &tc, prof, ws, ws_bytes, &res->tls, st, true, &tp, guide_ready, s_clean));
     res->tls_w_max = tp.path == 7 ? 32 : rec == JP_TLS_ONCHIP ? tp.window : wm;
@@ -1560,6 +1650,8 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
   // the classify pass also writes the TLS guide bitmaps when the loop can be guided
   // (A read through an index, workspace with the guide region): no separate guide pass
   int clean = 0;
+  int64_t dist[32];
+  bool have_dist = false;
   cudaEvent_t vdone = nullptr;
   // every exit (an error return included) orders st after the side-stream clear
   // of the shadow values and releases the event
@@ -1587,10 +1679,12 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
     else JP_TRY(jp_profile_stamp(L, ws, ws_bytes, stp));
     JP_CUDA(launch_prof_classify_guide(j, ws, lg, st, pairs), "profile classify");
     join_v.join();   // everything after the profile on st (TLS, or any later call) sees V zeroed
-    int64_t h[8];
+    int64_t h[H_DIST + 32];
     JP_CUDA(d2h_small_sync(h, at<int64_t>(ws, lg, R_HEADER), sizeof h, st), "profile D2H");
     if (h[H_BAD]) return fail(JP_ERR_INDEX, "%lld index entries are outside their arrays", (long long)h[H_BAD]);
     fill_profile(&p, L->n, h);
+    memcpy(dist, h + H_DIST, sizeof dist);
+    have_dist = true;
   } else {
     JP_TRY(jp_profile_density(L, ws, ws_bytes, nullptr, 0, nullptr, &p, stp));
   }
@@ -1599,7 +1693,8 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
   res->mode = select_mode_counts(p.n, p.raw_iters, p.war_iters, p.waw_iters, c.tau_high);
   res->n_tasks = 1;
   res->n_batches = 1;
-  return run_mode(L, j, res->mode, &p, c, ws, ws_bytes, res, st, gfuse && p.waw_iters == 0, clean);
+  return run_mode(L, j, res->mode, &p, c, ws, ws_bytes, res, st, gfuse && p.waw_iters == 0, clean,
+                  have_dist ? dist : nullptr);
 }
 
 

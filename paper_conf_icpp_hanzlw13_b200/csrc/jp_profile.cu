@@ -194,7 +194,8 @@ __device__ __forceinline__ int2 pair32(const int2 *p, int32_t a, int32_t len) {
 // so a warp's 128 consecutive iterations of one quad step span at most two chunks
 template <int OP, bool GUIDE, bool PAIRS = false>
 __global__ void __launch_bounds__(256) k_prof_count4(DLoop L, Tabs t, int vec, int64_t *hdr, uint32_t *graw,
-                                                     uint32_t *gsrc, int64_t chunk = 0, int64_t *cc = nullptr) {
+                                                     uint32_t *gsrc, int64_t chunk = 0, int64_t *cc = nullptr,
+                                                     unsigned long long *dist = nullptr) {
   __shared__ unsigned long long s_cnt[3];
   __shared__ unsigned long long s_first;
   // PRIV_TMP with a small T (config 4: 1024 slots): its first-writer table in
@@ -216,11 +217,17 @@ __global__ void __launch_bounds__(256) k_prof_count4(DLoop L, Tabs t, int vec, i
   unsigned c_raw = 0, c_war = 0, c_waw = 0;
   unsigned long long first = ~0ull;
   const int64_t nq = (L.n + 3) >> 2, B = blockDim.x;
-  // the writer (local iteration) behind a raw read of address a: mark it a RAW source
-  auto mark_src = [&](int32_t a) {
+  // the writer (local iteration) behind a raw read of address a: mark it a RAW
+  // source, and count the read's dependence distance i - j (floor log2) for the
+  // restart-TLS window choice (jp_schedule, restart_plan)
+  __shared__ unsigned s_dist[GUIDE ? 32 : 1];
+  if (GUIDE && threadIdx.x < 32) s_dist[threadIdx.x] = 0;
+  auto mark_src = [&](int32_t a, int32_t e) {
     if constexpr (GUIDE) {
-      const int64_t j = (int64_t)(0x7FFFFFFF - (PAIRS ? t.pA[a].x : t.wA[a])) - L.base;
+      const int32_t we = PAIRS ? t.pA[a].x : t.wA[a];
+      const int64_t j = (int64_t)(0x7FFFFFFF - we) - L.base;
       atomicOr(&gsrc[j >> 5], 1u << (j & 31));
+      if (dist) atomicAdd(&s_dist[31 - __clz(we - e)], 1u);
     }
   };
   for (int64_t q0 = (int64_t)blockIdx.x * B * kQuadSteps + threadIdx.x; q0 - threadIdx.x < nq; q0 += (int64_t)gridDim.x * B * kQuadSteps) {
@@ -263,7 +270,7 @@ __global__ void __launch_bounds__(256) k_prof_count4(DLoop L, Tabs t, int vec, i
               waw = earlier32(t.wA, a, lenA, e);
             }
             raw = b == a ? waw : PAIRS ? pair32(t.pA, b, lenA).x > e : earlier32(t.wA, b, lenA, e);
-            if (raw) mark_src(b);
+            if (raw) mark_src(b, e);
           } else if constexpr (OP == JP_OP_SAXPY) {
             if constexpr (PAIRS) {
               const int2 pa = pair32(t.pA, a, lenA);
@@ -274,7 +281,7 @@ __global__ void __launch_bounds__(256) k_prof_count4(DLoop L, Tabs t, int vec, i
               war = earlier32(t.rA, a, lenA, e);
             }
             waw = raw;
-            if (raw) mark_src(a);
+            if (raw) mark_src(a, e);
           } else if constexpr (OP == JP_OP_PRIV_TMP) {
             war = earlier32(rT, a, lenT, e);
             waw = earlier32(wT, a, lenT, e) || earlier32(t.wA, q4(vb[u], k), lenA, e);
@@ -291,8 +298,8 @@ __global__ void __launch_bounds__(256) k_prof_count4(DLoop L, Tabs t, int vec, i
             const bool r0 = b == a ? waw : PAIRS ? pair32(t.pA, b, lenA).x > e : earlier32(t.wA, b, lenA, e);
             const bool r1 = c == a ? waw : c == b ? r0 : PAIRS ? pair32(t.pA, c, lenA).x > e : earlier32(t.wA, c, lenA, e);
             raw = r0 || r1;
-            if (r0) mark_src(q4(vb[u], k));
-            if (r1) mark_src(q4(vc[u], k));
+            if (r0) mark_src(q4(vb[u], k), e);
+            if (r1) mark_src(q4(vc[u], k), e);
           }
           c_raw += raw; c_war += war; c_waw += waw;
           qr += raw; qa += war; qw += waw;
@@ -342,6 +349,9 @@ __global__ void __launch_bounds__(256) k_prof_count4(DLoop L, Tabs t, int vec, i
   JP_CTA_SYNC();
   if (threadIdx.x < 3 && s_cnt[threadIdx.x]) atomicAdd((unsigned long long *)&hdr[H_RAW + threadIdx.x], s_cnt[threadIdx.x]);
   if (threadIdx.x == 0 && s_first != ~0ull) atomicMin((unsigned long long *)&hdr[H_FIRST_RAW], s_first);
+  if constexpr (GUIDE) {
+    if (dist && threadIdx.x < 32 && s_dist[threadIdx.x]) atomicAdd(&dist[threadIdx.x], (unsigned long long)s_dist[threadIdx.x]);
+  }
 }
 
 static int idx_vec(const DLoop &d) {
@@ -791,6 +801,7 @@ static void run_classify_guide(const DLoop &d, Tabs t, uint32_t *graw, uint32_t 
   (void)DT;
   const int64_t nq = (d.n + 3) / 4;
   const int g = grid_for((nq + kQuadSteps - 1) / kQuadSteps, 256, 8);
+  auto *dist = reinterpret_cast<unsigned long long *>(hdr + H_DIST);
   if constexpr (OP == JP_OP_PRIV_TMP) {   // never guided: counts only
     k_prof_count4<OP, false><<<g, 256, 0, st>>>(d, t, idx_vec(d), hdr, nullptr, nullptr);
   } else {
@@ -799,9 +810,9 @@ static void run_classify_guide(const DLoop &d, Tabs t, uint32_t *graw, uint32_t 
         k_interleave<<<grid_for(d.lenA / 4 + 1, 256, 8), 256, 0, st>>>(t.wA, t.rA, const_cast<int2 *>(t.pA), d.lenA);
         note_launch();
       }
-      k_prof_count4<OP, true, true><<<g, 256, 0, st>>>(d, t, idx_vec(d), hdr, graw, gsrc);
+      k_prof_count4<OP, true, true><<<g, 256, 0, st>>>(d, t, idx_vec(d), hdr, graw, gsrc, 0, nullptr, dist);
     } else {
-      k_prof_count4<OP, true><<<g, 256, 0, st>>>(d, t, idx_vec(d), hdr, graw, gsrc);
+      k_prof_count4<OP, true><<<g, 256, 0, st>>>(d, t, idx_vec(d), hdr, graw, gsrc, 0, nullptr, dist);
     }
   }
   note_launch();
@@ -813,6 +824,7 @@ cudaError_t launch_prof_classify_guide(const Job &j, void *ws, const Layout &lo,
   if (!bits) return launch_prof_classify(j, ws, lo, nullptr, 0, nullptr, st);
   cudaMemsetAsync(&hdr[H_RAW], 0, 3 * sizeof(int64_t), st);
   cudaMemsetAsync(&hdr[H_FIRST_RAW], 0xFF, sizeof(int64_t), st);
+  cudaMemsetAsync(&hdr[H_DIST], 0, 32 * sizeof(int64_t), st);
   const int64_t nw = (j.d.n + 31) / 32;
   cudaMemsetAsync(bits + nw, 0, 4 * (size_t)nw, st);   // source words are OR-ed in
   if (j.d.n == 0) return launch_check();

@@ -41,6 +41,7 @@ def main():
     ap = argparse.ArgumentParser()
     ap.add_argument("--n", type=int, default=22)
     ap.add_argument("--skip-fixed", action="store_true")
+    ap.add_argument("--schedule-only", action="store_true")
     args = ap.parse_args()
     st = torch.cuda.current_stream()
     dev = torch.device("cuda:0")
@@ -72,6 +73,15 @@ def main():
                 L = jp.Loop.from_workload(wl)
                 ws = jp.workspace(L)
                 prof = jp.jp_profile_density(L, ws)
+                for rec in (1, 0):
+                    res, ms = timed(lambda: jp.jp_schedule(L, ws, stream=st, tls_recovery=rec), wl.A, A0, st, reps=1)
+                    print(json.dumps({"loop": tag, "d": d, "delta": delta, "schedule": rec, "ms": ms,
+                                      "G_committed_per_s": n / ms / 1e6, "mode": res["mode_name"],
+                                      "path": res["tls_path"], "w_max": res["tls_w_max"],
+                                      "recovery": res["tls_recovery"], "windows": res["tls"]["windows"],
+                                      "violations": res["tls"]["violations"]}), flush=True)
+                if args.schedule_only:
+                    continue
                 for path, wm in ((1, 256), (1, 1024), (1, 4096), (3, 4096), (3, 16384), (3, 65536), (2, 65536),
                                  (2, 262144)):
                     try:
