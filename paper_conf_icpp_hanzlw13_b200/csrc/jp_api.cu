@@ -1584,14 +1584,14 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
       Layout lo;
       JP_TRY(check_ws(L, ws, ws_bytes, smode == JP_MODE_PRIVATIZED ? JP_WS_PRIV : 0, lo));
       int64_t *bad = &at<int64_t>(ws, lo, R_HEADER)[H_BAD];
-      JP_CUDA(launch_validate_indirect(j, bad, st), "validate");
       Job jr = j;
       jr.d.abort = bad;
       if (smode == JP_MODE_PRIVATIZED) {
         bool applied = false;
-        JP_CUDA(launch_priv_stream(jr, ws, lo, true, st, 0, true, &applied), "priv stream");
+        JP_CUDA(launch_priv_stream(jr, ws, lo, true, st, 0, true, &applied, bad), "priv stream");
         if (!applied) JP_CUDA(launch_priv_finalize(jr, ws, lo, st), "priv finalize");
       } else {
+        JP_CUDA(launch_validate_indirect(j, bad, st), "validate");
         JP_CUDA(launch_doall(jr, st), "doall");
       }
       int64_t nb = 0;

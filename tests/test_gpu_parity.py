@@ -160,8 +160,8 @@ def test_index_error_no_side_effects():
     assert jp.jp_validate(L, ws) == 1
 
 
-@pytest.mark.parametrize("case", ["c4", "c4_w", "saxpy_r"])
-def test_structural_raw_free_schedule(case):
+@pytest.mark.parametrize("case", ["c4", "c4_w", "saxpy_r", "c4_tail"])
+def test_structural_raw_free_schedule(case, doall_kernel):
     """Reading B11: PRIV_TMP (X read-only, T's read covered) and SAXPY with
     identity writes are run without a profile (profiled = 0) -- results equal the
     oracle; an out-of-range indirect index gives JP_ERR_INDEX with every array
@@ -169,6 +169,9 @@ def test_structural_raw_free_schedule(case):
     n = (1 << 20) + 77
     g0 = np.random.default_rng(3)
     if case == "c4":
+        wl, mode = synth.config4(n=n), jp.JP_MODE_PRIVATIZED
+    elif case == "c4_tail":   # one 4096-iteration tile and a ragged element tail (beyond the tiny path)
+        n = 4096 + 3001
         wl, mode = synth.config4(n=n), jp.JP_MODE_PRIVATIZED
     elif case == "c4_w":   # Y written through a 2-to-1 index: WAW on Y as well
         wl, mode = synth.config4(n=n), jp.JP_MODE_PRIVATIZED
