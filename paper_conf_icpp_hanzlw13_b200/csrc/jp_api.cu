@@ -1246,9 +1246,15 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
   // the first all-SM TLS task finds this call's pair table in the write-log
   // region: it needs no reset (see launch_tls_fwd_grid); later ones do
   bool s_fresh = pairs;
-  JP_CUDA(launch_prof_stamp(j, ws, lo, st, pairs), "profile stamp");
-  JP_CUDA(launch_prof_classify(j, ws, lo, gbits, chunk, cc, st, gbits ? gbits + (L->n + 31) / 32 : nullptr, pairs),
-          "profile classify");
+  if (bucket_profile_ok(j, ws, lo)) {   // large A: the profile by address buckets (jp_bucket.cu)
+    s_fresh = false;                    // (region 7 is not filled: the TLS task resets it)
+    JP_CUDA(launch_prof_bucket(j, ws, lo, gbits, gbits ? gbits + (L->n + 31) / 32 : nullptr, chunk, cc, st),
+            "profile (buckets)");
+  } else {
+    JP_CUDA(launch_prof_stamp(j, ws, lo, st, pairs), "profile stamp");
+    JP_CUDA(launch_prof_classify(j, ws, lo, gbits, chunk, cc, st, gbits ? gbits + (L->n + 31) / 32 : nullptr, pairs),
+            "profile classify");
+  }
   std::vector<int64_t> hc(3 * nck), h(8);
   JP_CUDA(cudaMemcpyAsync(hc.data(), cc, 24 * nck, cudaMemcpyDeviceToHost, st), "chunk D2H");
   JP_CUDA(cudaMemcpyAsync(h.data(), at<int64_t>(ws, lo, R_HEADER), 64, cudaMemcpyDeviceToHost, st), "profile D2H");
@@ -1674,10 +1680,16 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
       cudaEventRecord(vdone, side);
       clean = 2;
     }
-    if (pairs) clean |= 1;
-    if (pairs) JP_CUDA(launch_prof_stamp(j, ws, lg, st, true, pairs_ready), "profile stamp");
-    else JP_TRY(jp_profile_stamp(L, ws, ws_bytes, stp));
-    JP_CUDA(launch_prof_classify_guide(j, ws, lg, st, pairs), "profile classify");
+    if (pairs) clean |= 1;   // region 7 holds this call's pair table, or the side stream's all-ones fill
+    if (bucket_profile_ok(j, ws, lg)) {
+      // large A: the profile by address buckets (jp_bucket.cu), guide words included
+      uint32_t *g = at<uint32_t>(ws, lg, R_GUIDE);
+      JP_CUDA(launch_prof_bucket(j, ws, lg, g, g + (L->n + 31) / 32, 0, nullptr, st), "profile (buckets)");
+    } else {
+      if (pairs) JP_CUDA(launch_prof_stamp(j, ws, lg, st, true, pairs_ready), "profile stamp");
+      else JP_TRY(jp_profile_stamp(L, ws, ws_bytes, stp));
+      JP_CUDA(launch_prof_classify_guide(j, ws, lg, st, pairs), "profile classify");
+    }
     join_v.join();   // everything after the profile on st (TLS, or any later call) sees V zeroed
     int64_t h[H_DIST + 32];
     JP_CUDA(d2h_small_sync(h, at<int64_t>(ws, lg, R_HEADER), sizeof h, st), "profile D2H");

@@ -1,0 +1,470 @@
+// jp_bucket.cu -- the dependency-density profile of a loop over a large A by
+// address buckets (P1 stamp + P2 classify of SURVEY Sec.8(a); the paper's
+// profiler, Fig. 1 "DD analysis"; densities per reading A1).
+//
+// The two-pass stamp/classify profile (jp_profile.cu) needs one random L2 atomic
+// per access (first writer / first reader of the address) and then random reads
+// of the same tables: on config 3 (N = len_A = 2^24) that is 2^25 atomics at the
+// L2 atomic rate (3 address-window passes) plus a classify pass whose lookups
+// miss L2 -- 1.6 GB of DRAM traffic for 0.47 GB of algorithmic bytes.  Here the
+// accesses are first PARTITIONED by address instead, so every first-writer /
+// first-reader table lives in one CTA's shared memory:
+//
+//   count    per tile of 4096 iterations: accesses per bucket of 8192
+//            addresses (shared-memory histogram), and the out-of-range count;
+//   scan     per bucket, the tiles' exclusive offsets; then the buckets' bases;
+//   scatter  every access as an 8-byte record (iteration, address in its
+//            bucket, write / read) into its bucket's segment, tile by tile:
+//            staged in shared memory grouped by bucket first, so each (tile,
+//            bucket) run is written as one contiguous piece (random 4-byte
+//            stores were bound by L2 transactions: 345 us on config 3);
+//   evaluate one CTA per bucket: minW / minR of its 8192 addresses by shared
+//            atomics over the bucket's records, then every record evaluated
+//            against them -- raw (an exposed read whose first writer is
+//            earlier), war / waw (a write whose first reader / writer is
+//            earlier) -- with the per-iteration guide bits, the RAW-source bits
+//            (the first writer of every raw read), the raw-distance histogram,
+//            the first raw iteration and optional per-chunk counts.
+//
+// DRAM traffic per iteration (ADD_C): index streams twice (16 B), records
+// written and read once (2 x 2 x 8 B); the tables never leave shared memory.
+// (4-byte records holding the iteration within its tile were measured slower:
+// recovering the tile of every record costs more instructions than the bytes.)
+// Counts are per access: ADD_C has exactly one write and one exposed read of A
+// per iteration (raw from the read, war / waw from the write); SAXPY's only A
+// access is Y[w], read and written by the same iteration, so raw = war = waw =
+// "an earlier iteration wrote this address" (one write record).
+#include "jp_host.h"
+
+namespace jp {
+
+constexpr int kBShift = 13;                 // addresses per bucket: 8192
+constexpr int kBSpan = 1 << kBShift;
+constexpr int kTShift = 12;                 // iterations per tile: 4096
+constexpr int kTile = 1 << kTShift;
+constexpr int kBThreads = 512;
+constexpr int kEvalThreads = 512;
+constexpr int kMaxBuckets = 8192;           // len_A <= 2^26
+constexpr int kMaxTiles = 16384;            // n <= 2^26
+constexpr int kSmemChunks = 1024;           // per-chunk counts kept in shared memory up to this many chunks
+// record (8 bytes): local iteration (low word) | address in the bucket << 32 | write << 63
+constexpr unsigned long long kRecW = 1ull << 63;
+
+struct BkView {
+  const int32_t *r, *w;   // ADD_C: read r, write w; SAXPY: w only (NULL => identity ioff + i)
+  int64_t n, ioff;
+  uint32_t lenA;
+  int B, T;
+};
+
+__device__ __forceinline__ int4 ld_idx4(const int32_t *p, int64_t i, int64_t n, int64_t ioff, bool vec) {
+  if (!p) {
+    const int b = (int)(ioff + i);
+    return make_int4(b, b + 1, b + 2, b + 3);
+  }
+  if (vec && i + 4 <= n) return __ldcs(reinterpret_cast<const int4 *>(p + i));
+  int4 v;
+  v.x = p[i];
+  v.y = i + 1 < n ? p[i + 1] : 0;
+  v.z = i + 2 < n ? p[i + 2] : 0;
+  v.w = i + 3 < n ? p[i + 3] : 0;
+  return v;
+}
+__device__ __forceinline__ int q4(const int4 &v, int k) { return k == 0 ? v.x : k == 1 ? v.y : k == 2 ? v.z : v.w; }
+
+// Visit the accesses of tile blockIdx.x four iterations at a time (16-byte
+// index loads, kU quads in flight per lane): f(a[8], wr[8], il0, kn) gets the
+// quad's accesses -- ADD_C: (w, r) of each of the kn <= 4 iterations, SAXPY: w.
+template <int OP, typename F>
+__device__ __forceinline__ void for_tile(const BkView &V, bool vec, F &&f) {
+  const int64_t t0 = (int64_t)blockIdx.x << kTShift;
+  const int64_t tn = V.n - t0 < kTile ? V.n - t0 : kTile;
+  const int nq = (int)((tn + 3) >> 2);
+  constexpr int kU = 4;
+  for (int q0 = threadIdx.x; q0 < nq; q0 += kBThreads * kU) {
+    int4 vw[kU], vr[kU];
+#pragma unroll
+    for (int u = 0; u < kU; u++) {
+      const int q = q0 + u * kBThreads;
+      if (q < nq) {
+        vw[u] = ld_idx4(V.w, t0 + 4 * q, V.n, V.ioff, vec);
+        if constexpr (OP == JP_OP_ADD_C) vr[u] = ld_idx4(V.r, t0 + 4 * q, V.n, V.ioff, vec);
+      }
+    }
+#pragma unroll
+    for (int u = 0; u < kU; u++) {
+      const int q = q0 + u * kBThreads;
+      if (q >= nq) break;
+      const int kn = tn - 4 * q < 4 ? (int)(tn - 4 * q) : 4;
+      f(vw[u], vr[u], 4 * q, kn);
+    }
+  }
+}
+
+// cnt[t * B + b] = accesses of tile t into bucket b; out-of-range indices counted into *bad
+template <int OP>
+__global__ void __launch_bounds__(kBThreads) k_bk_count(BkView V, int vec, uint32_t *cnt, int64_t *bad) {
+  extern __shared__ uint32_t h[];
+  for (int b = threadIdx.x; b < V.B; b += kBThreads) h[b] = 0;
+  __syncthreads();
+  unsigned nbad = 0;
+  // an out-of-range index is counted (the profile then fails) and filed under
+  // bucket 0, consistently with the scatter below
+  for_tile<OP>(V, vec, [&](const int4 &w4, const int4 &r4, int, int kn) {
+#pragma unroll
+    for (int k = 0; k < 4; k++) {
+      if (k < kn) {
+        const uint32_t a = (uint32_t)q4(w4, k);
+        nbad += a >= V.lenA;
+        atomicAdd(&h[a < V.lenA ? a >> kBShift : 0], 1u);
+        if constexpr (OP == JP_OP_ADD_C) {
+          const uint32_t c = (uint32_t)q4(r4, k);
+          nbad += c >= V.lenA;
+          atomicAdd(&h[c < V.lenA ? c >> kBShift : 0], 1u);
+        }
+      }
+    }
+  });
+  nbad = __reduce_add_sync(0xffffffffu, nbad);
+  if ((threadIdx.x & 31) == 0 && nbad) atomicAdd(reinterpret_cast<unsigned long long *>(bad), (unsigned long long)nbad);
+  __syncthreads();
+  uint32_t *row = cnt + (size_t)blockIdx.x * V.B;
+  for (int b = threadIdx.x; b < V.B; b += kBThreads) row[b] = h[b];
+}
+
+// per bucket: exclusive prefix over the tiles (in place) and the bucket total.
+// Block = 32 buckets (one per lane) x 32 tile segments (one per warp).
+__global__ void __launch_bounds__(1024) k_bk_scan_tiles(uint32_t *cnt, int T, int B, uint32_t *tot) {
+  __shared__ uint32_t part[32][33];
+  const int lane = threadIdx.x & 31, seg = threadIdx.x >> 5;
+  const int b = blockIdx.x * 32 + lane;
+  const int per = (T + 31) / 32, t0 = seg * per, t1 = min(T, t0 + per);
+  uint32_t s = 0;
+  if (b < B)
+#pragma unroll 8
+    for (int t = t0; t < t1; t++) s += cnt[(size_t)t * B + b];
+  part[seg][lane] = s;
+  __syncthreads();
+  uint32_t run = 0;
+  for (int k = 0; k < seg; k++) run += part[k][lane];
+  if (b < B) {
+#pragma unroll 8
+    for (int t = t0; t < t1; t++) {
+      const uint32_t v = cnt[(size_t)t * B + b];
+      cnt[(size_t)t * B + b] = run;
+      run += v;
+    }
+    if (seg == 31) tot[b] = run;
+  }
+}
+
+// base[b] = exclusive prefix of tot over the buckets (one CTA)
+__global__ void __launch_bounds__(1024) k_bk_scan_buckets(const uint32_t *tot, int B, uint32_t *base) {
+  __shared__ uint32_t ws[32];
+  const int per = (B + 1023) / 1024, b0 = threadIdx.x * per;
+  uint32_t s = 0;
+  for (int k = 0; k < per && b0 + k < B; k++) s += tot[b0 + k];
+  uint32_t x = s;   // inclusive warp scan
+  for (int o = 1; o < 32; o <<= 1) {
+    const uint32_t y = __shfl_up_sync(0xffffffffu, x, o);
+    if ((threadIdx.x & 31) >= o) x += y;
+  }
+  if ((threadIdx.x & 31) == 31) ws[threadIdx.x >> 5] = x;
+  __syncthreads();
+  if (threadIdx.x < 32) {
+    uint32_t v = ws[threadIdx.x];
+    for (int o = 1; o < 32; o <<= 1) {
+      const uint32_t y = __shfl_up_sync(0xffffffffu, v, o);
+      if (threadIdx.x >= o) v += y;
+    }
+    ws[threadIdx.x] = v;
+  }
+  __syncthreads();
+  uint32_t run = x - s + ((threadIdx.x >> 5) ? ws[(threadIdx.x >> 5) - 1] : 0);
+  for (int k = 0; k < per && b0 + k < B; k++) {
+    base[b0 + k] = run;
+    run += tot[b0 + k];
+  }
+}
+
+// records, tile-ordered inside each bucket's segment.  Shared memory: the
+// tile's records staged by bucket (2 x 16384 x 4 B), the local bucket starts
+// and cursors (B each), the global start of this tile's run in every bucket.
+template <int OP>
+__global__ void __launch_bounds__(kBThreads) k_bk_scatter(BkView V, int vec, const uint32_t *off, const uint32_t *tot,
+                                                         const uint32_t *base, unsigned long long *rec) {
+  extern __shared__ unsigned long long sm64[];
+  unsigned long long *stage = sm64;                            // [2 * kTile] il | a << 12 | write << 63
+  uint32_t *lpos = reinterpret_cast<uint32_t *>(stage + 2 * kTile);   // [B + 1] local exclusive starts
+  uint32_t *cur = lpos + V.B + 1;                              // [B]
+  uint32_t *gpos = cur + V.B;                                  // [B] global start of this tile's run
+  __shared__ uint32_t wsum[kBThreads / 32];
+  const int t = blockIdx.x, B = V.B;
+  const uint32_t i0 = (uint32_t)t << kTShift;
+  const uint32_t *row = off + (size_t)t * B, *nxt = t + 1 < V.T ? row + B : nullptr;
+  // local counts -> exclusive scan over the buckets (per thread a contiguous run)
+  const int per = (B + kBThreads - 1) / kBThreads, b0 = threadIdx.x * per;
+  uint32_t s = 0;
+  for (int k = 0; k < per && b0 + k < B; k++) {
+    const int b = b0 + k;
+    const uint32_t c = (nxt ? nxt[b] : tot[b]) - row[b];
+    cur[b] = c;   // (count, for the scan below)
+    gpos[b] = base[b] + row[b];
+    s += c;
+  }
+  uint32_t x = s;
+  for (int o = 1; o < 32; o <<= 1) {
+    const uint32_t y = __shfl_up_sync(0xffffffffu, x, o);
+    if ((threadIdx.x & 31) >= o) x += y;
+  }
+  if ((threadIdx.x & 31) == 31) wsum[threadIdx.x >> 5] = x;
+  __syncthreads();
+  uint32_t wpre = 0;
+  for (int k = 0; k < (int)(threadIdx.x >> 5); k++) wpre += wsum[k];
+  uint32_t run = wpre + x - s;
+  for (int k = 0; k < per && b0 + k < B; k++) {
+    const int b = b0 + k;
+    const uint32_t c = cur[b];
+    lpos[b] = run;
+    cur[b] = run;
+    run += c;
+  }
+  if (threadIdx.x == kBThreads - 1) lpos[B] = run;
+  __syncthreads();
+  for_tile<OP>(V, vec, [&](const int4 &w4, const int4 &r4, int il0, int kn) {
+    // all positions of the quad first (the shared atomics issue back to back),
+    // then the staging stores
+    constexpr int kA = OP == JP_OP_ADD_C ? 8 : 4;
+    uint32_t a[kA], pos[kA];
+#pragma unroll
+    for (int k = 0; k < 4; k++) {
+      a[OP == JP_OP_ADD_C ? 2 * k : k] = (uint32_t)q4(w4, k);
+      if constexpr (OP == JP_OP_ADD_C) a[2 * k + 1] = (uint32_t)q4(r4, k);
+    }
+#pragma unroll
+    for (int m = 0; m < kA; m++) {
+      if (a[m] >= V.lenA) a[m] = 0;   // (the count pass filed it under bucket 0 too)
+      const int k = OP == JP_OP_ADD_C ? m >> 1 : m;
+      pos[m] = k < kn ? atomicAdd(&cur[a[m] >> kBShift], 1u) : 0u;
+    }
+#pragma unroll
+    for (int m = 0; m < kA; m++) {
+      const int k = OP == JP_OP_ADD_C ? m >> 1 : m;
+      const bool wr = OP == JP_OP_ADD_C ? (m & 1) == 0 : true;
+      if (k < kn)
+        stage[pos[m]] = (unsigned long long)(il0 + k) | (unsigned long long)a[m] << kTShift | (wr ? kRecW : 0ull);
+    }
+  });
+  __syncthreads();
+  // copy out, flat: staged record k of bucket b goes to k + (gpos[b] - lpos[b])
+  // (consecutive k of one run are consecutive records of the bucket's segment)
+  for (int b = threadIdx.x; b < B; b += kBThreads) gpos[b] -= lpos[b];
+  __syncthreads();
+  const uint32_t nrec = lpos[B];
+  for (uint32_t k = threadIdx.x; k < nrec; k += kBThreads) {
+    const unsigned long long x = stage[k];
+    const uint32_t a = (uint32_t)(x >> kTShift) & 0x7FFFFFFFu;
+    rec[k + gpos[a >> kBShift]] = (unsigned long long)(i0 + ((uint32_t)x & (kTile - 1))) |
+                                  (unsigned long long)(a & (kBSpan - 1)) << 32 | (x & kRecW);
+  }
+}
+
+struct BkOut {
+  int64_t *hdr;               // H_RAW / H_WAR / H_WAW, H_FIRST_RAW, H_DIST
+  uint32_t *graw, *gsrc;      // guide words (nullable), zeroed by the caller
+  int64_t chunk;              // per-chunk counts (cc nullable)
+  int64_t *cc;
+  int64_t gbase;              // global id of local iteration 0
+};
+
+template <int OP>
+__global__ void __launch_bounds__(kEvalThreads) k_bk_eval(BkView V, const uint32_t *base, const uint32_t *tot,
+                                                          const unsigned long long *rec, BkOut O) {
+  // dynamic: minW[8192], minR[8192] (ADD_C), then 3 x nch per-chunk counts when they fit
+  extern __shared__ uint32_t s_dyn[];
+  uint32_t *minW = s_dyn;
+  uint32_t *minR = s_dyn + kBSpan;
+  uint32_t *s_cc = s_dyn + (OP == JP_OP_ADD_C ? 2 : 1) * kBSpan;
+  __shared__ unsigned s_dist[32];
+  __shared__ unsigned long long s_cnt[3], s_first;
+  const int b = blockIdx.x;
+  const int nch = O.cc ? (int)((V.n + O.chunk - 1) / O.chunk) : 0;
+  const bool cc_smem = O.cc && nch <= kSmemChunks;
+  for (int k = threadIdx.x; k < kBSpan; k += kEvalThreads) {
+    minW[k] = 0xFFFFFFFFu;
+    if constexpr (OP == JP_OP_ADD_C) minR[k] = 0xFFFFFFFFu;
+  }
+  const uint32_t total = tot[b];
+  if (threadIdx.x < 32) s_dist[threadIdx.x] = 0;
+  if (threadIdx.x < 3) s_cnt[threadIdx.x] = 0;
+  if (threadIdx.x == 0) s_first = ~0ull;
+  if (cc_smem)
+    for (int k = threadIdx.x; k < 3 * nch; k += kEvalThreads) s_cc[k] = 0;
+  __syncthreads();
+  const unsigned long long *rb = rec + base[b];
+  constexpr int kU = 4;   // records in flight per thread
+  auto sweep = [&](auto &&f) {
+    for (uint32_t p0 = threadIdx.x; p0 < total; p0 += kEvalThreads * kU) {
+      unsigned long long xv[kU];
+#pragma unroll
+      for (int u = 0; u < kU; u++) {
+        const uint32_t p = p0 + (uint32_t)u * kEvalThreads;
+        xv[u] = p < total ? rb[p] : 0ull;
+      }
+#pragma unroll
+      for (int u = 0; u < kU; u++)
+        if (p0 + (uint32_t)u * kEvalThreads < total) f(xv[u]);
+    }
+  };
+  // pass 1: first writer / first reader of every address of the bucket
+  sweep([&](unsigned long long x) {
+    const uint32_t i = (uint32_t)x, al = (uint32_t)(x >> 32) & (kBSpan - 1);
+    if (x & kRecW) atomicMin(&minW[al], i);
+    else if constexpr (OP == JP_OP_ADD_C) atomicMin(&minR[al], i);
+  });
+  __syncthreads();
+  // pass 2: every access against the final tables
+  unsigned c_raw = 0, c_war = 0, c_waw = 0;
+  unsigned long long first = ~0ull;
+  sweep([&](unsigned long long x) {
+    const uint32_t i = (uint32_t)x, al = (uint32_t)(x >> 32) & (kBSpan - 1);
+    const uint32_t jw = minW[al];
+    bool raw, war = false, waw = false;
+    if (x & kRecW) {
+      waw = jw < i;
+      war = (OP == JP_OP_ADD_C ? minR[al] : jw) < i;
+      raw = OP == JP_OP_SAXPY && waw;
+    } else {
+      raw = jw < i;
+    }
+    c_raw += raw; c_war += war; c_waw += waw;
+    if (raw) {
+      if (O.graw) atomicOr(&O.graw[i >> 5], 1u << (i & 31));
+      if (O.gsrc) atomicOr(&O.gsrc[jw >> 5], 1u << (jw & 31));
+      atomicAdd(&s_dist[31 - __clz(i - jw)], 1u);
+      if ((unsigned long long)i < first) first = i;
+    }
+    if (O.cc && (raw | war | waw)) {
+      const int64_t ch = (int64_t)i / O.chunk;
+      if (cc_smem) {
+        if (raw) atomicAdd(&s_cc[3 * ch + 0], 1u);
+        if (war) atomicAdd(&s_cc[3 * ch + 1], 1u);
+        if (waw) atomicAdd(&s_cc[3 * ch + 2], 1u);
+      } else {
+        if (raw) atomicAdd(reinterpret_cast<unsigned long long *>(&O.cc[3 * ch + 0]), 1ull);
+        if (war) atomicAdd(reinterpret_cast<unsigned long long *>(&O.cc[3 * ch + 1]), 1ull);
+        if (waw) atomicAdd(reinterpret_cast<unsigned long long *>(&O.cc[3 * ch + 2]), 1ull);
+      }
+    }
+  });
+  c_raw = __reduce_add_sync(0xffffffffu, c_raw);
+  c_war = __reduce_add_sync(0xffffffffu, c_war);
+  c_waw = __reduce_add_sync(0xffffffffu, c_waw);
+  for (int o = 16; o; o >>= 1) {
+    const unsigned long long y = __shfl_xor_sync(0xffffffffu, first, o);
+    first = y < first ? y : first;
+  }
+  if ((threadIdx.x & 31) == 0) {
+    if (c_raw) atomicAdd(&s_cnt[0], (unsigned long long)c_raw);
+    if (c_war) atomicAdd(&s_cnt[1], (unsigned long long)c_war);
+    if (c_waw) atomicAdd(&s_cnt[2], (unsigned long long)c_waw);
+    if (first != ~0ull) atomicMin(&s_first, first);
+  }
+  __syncthreads();
+  if (threadIdx.x < 3 && s_cnt[threadIdx.x])
+    atomicAdd(reinterpret_cast<unsigned long long *>(&O.hdr[H_RAW + threadIdx.x]), s_cnt[threadIdx.x]);
+  if (threadIdx.x == 0 && s_first != ~0ull)
+    atomicMin(reinterpret_cast<unsigned long long *>(&O.hdr[H_FIRST_RAW]), (unsigned long long)O.gbase + s_first);
+  if (threadIdx.x < 32 && s_dist[threadIdx.x])
+    atomicAdd(reinterpret_cast<unsigned long long *>(&O.hdr[H_DIST + threadIdx.x]), (unsigned long long)s_dist[threadIdx.x]);
+  if (cc_smem)
+    for (int k = threadIdx.x; k < 3 * nch; k += kEvalThreads)
+      if (s_cc[k]) atomicAdd(reinterpret_cast<unsigned long long *>(&O.cc[k]), (unsigned long long)s_cc[k]);
+}
+
+namespace {
+struct BkPlan {
+  BkView v;
+  unsigned long long *rec;
+  uint32_t *cnt, *tot, *base;
+};
+
+bool plan(const Job &j, void *ws, const Layout &lo, BkPlan &P) {
+  const DLoop &d = j.d;
+  if (!ws || d.n <= 0) return false;
+  if (j.op == JP_OP_ADD_C) {
+    if (!d.r && !d.w) return false;
+  } else if (j.op == JP_OP_SAXPY) {
+    if (!d.w) return false;
+  } else {
+    return false;
+  }
+  if (d.lenA < (1 << 20) || d.lenA > (int64_t)kMaxBuckets * kBSpan) return false;
+  if (d.n > (int64_t)kMaxTiles * kTile) return false;
+  const char *e = getenv("JP_PROFILE_BUCKETS");
+  if (e && e[0] == '0') return false;
+  const int B = (int)((d.lenA + kBSpan - 1) / kBSpan), T = (int)((d.n + kTile - 1) / kTile);
+  const int64_t nrec = (j.op == JP_OP_ADD_C ? 2 : 1) * d.n;
+  // records (8 B each) in minW_A .. keys_A when those regions are contiguous (the
+  // profile keeps no tables, and every privatized run clears the keys it
+  // applies); offsets in maxRx_A (free until a jp_tls_guide pass, which
+  // jp_schedule skips)
+  size_t rb = 0, endo = lo.off[R_MINW_A];
+  for (int r = R_MINW_A; r <= R_KEYS_A; r++) {
+    if (!lo.bytes[r]) continue;
+    if (lo.off[r] != endo) break;
+    rb += lo.bytes[r];
+    endo = lo.off[r] + lo.bytes[r];
+  }
+  if (!lo.bytes[R_MINW_A] || rb < 8 * (size_t)nrec) return false;
+  if (lo.bytes[R_MAXRX_A] < 4 * ((size_t)T * B + 2 * (size_t)B)) return false;
+  P.v = BkView{d.r, d.w, d.n, d.ioff, (uint32_t)d.lenA, B, T};
+  P.rec = at<unsigned long long>(ws, lo, R_MINW_A);
+  P.cnt = at<uint32_t>(ws, lo, R_MAXRX_A);
+  P.tot = P.cnt + (size_t)T * B;
+  P.base = P.tot + B;
+  return true;
+}
+
+template <int OP>
+void run_bucket(const BkPlan &P, const DLoop &d, int64_t *hdr, BkOut O, cudaStream_t st) {
+  auto al = [](const int32_t *q) { return q == nullptr || ((uintptr_t)q & 15) == 0; };
+  const int vec = al(d.r) && al(d.w);
+  const int B = P.v.B, T = P.v.T;
+  k_bk_count<OP><<<T, kBThreads, 4 * (size_t)B, st>>>(P.v, vec, P.cnt, &hdr[H_BAD]);
+  k_bk_scan_tiles<<<(B + 31) / 32, 1024, 0, st>>>(P.cnt, T, B, P.tot);
+  k_bk_scan_buckets<<<1, 1024, 0, st>>>(P.tot, B, P.base);
+  const size_t ssm = 8 * 2 * (size_t)kTile + 4 * (3 * (size_t)B + 1);
+  cudaFuncSetAttribute(k_bk_scatter<OP>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)ssm);
+  k_bk_scatter<OP><<<T, kBThreads, ssm, st>>>(P.v, vec, P.cnt, P.tot, P.base, P.rec);
+  const int nch = O.cc ? (int)((d.n + O.chunk - 1) / O.chunk) : 0;
+  const size_t sm = 4 * (size_t)kBSpan * (OP == JP_OP_ADD_C ? 2 : 1) + (O.cc && nch <= kSmemChunks ? 12 * (size_t)nch : 0);
+  cudaFuncSetAttribute(k_bk_eval<OP>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sm);
+  k_bk_eval<OP><<<B, kEvalThreads, sm, st>>>(P.v, P.base, P.tot, P.rec, O);
+  note_launch(5);
+}
+}  // namespace
+
+bool bucket_profile_ok(const Job &j, void *ws, const Layout &lo) {
+  BkPlan P;
+  return plan(j, ws, lo, P);
+}
+
+cudaError_t launch_prof_bucket(const Job &j, void *ws, const Layout &lo, uint32_t *graw, uint32_t *gsrc,
+                               int64_t chunk, int64_t *cc, cudaStream_t st) {
+  BkPlan P;
+  if (!plan(j, ws, lo, P)) return cudaErrorInvalidValue;
+  int64_t *hdr = at<int64_t>(ws, lo, R_HEADER);
+  cudaMemsetAsync(hdr, 0, kHeaderBytes, st);
+  cudaMemsetAsync(&hdr[H_FIRST_RAW], 0xFF, sizeof(int64_t), st);
+  const int64_t nw = (j.d.n + 31) / 32;
+  if (graw) cudaMemsetAsync(graw, 0, 4 * (size_t)nw, st);
+  if (gsrc) cudaMemsetAsync(gsrc, 0, 4 * (size_t)nw, st);
+  if (cc) cudaMemsetAsync(cc, 0, sizeof(int64_t) * 3 * ((j.d.n + chunk - 1) / chunk), st);
+  BkOut O{hdr, graw, gsrc, chunk, cc, j.d.base};
+  if (j.op == JP_OP_ADD_C) run_bucket<JP_OP_ADD_C>(P, j.d, hdr, O, st);
+  else run_bucket<JP_OP_SAXPY>(P, j.d, hdr, O, st);
+  return launch_check();
+}
+
+}  // namespace jp

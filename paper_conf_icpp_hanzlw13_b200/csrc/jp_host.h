@@ -54,6 +54,13 @@ cudaError_t launch_tls_guide(const Job &j, void *ws, const Layout &lo, cudaStrea
 cudaError_t launch_prof_stamp(const Job &j, void *ws, const Layout &lo, cudaStream_t st, bool pairs = false,
                               bool pairs_ready = false);
 bool stamp_pairs_ok(const Job &j, void *ws, const Layout &lo);
+// the profile by address buckets (jp_bucket.cu): counts, first raw, raw-distance
+// histogram, optional guide words (zeroed here) and per-chunk counts, for ADD_C /
+// SAXPY loops over a large A; uses minW/minR_A and maxRx_A as scratch (their
+// tables are NOT left filled).  bucket_profile_ok says whether it applies.
+bool bucket_profile_ok(const Job &j, void *ws, const Layout &lo);
+cudaError_t launch_prof_bucket(const Job &j, void *ws, const Layout &lo, uint32_t *graw, uint32_t *gsrc,
+                               int64_t chunk, int64_t *cc, cudaStream_t st);
 // src_bits (nullable): also the TLS guide's RAW-source words (raw_bits then holds its raw words)
 cudaError_t launch_prof_classify(const Job &j, void *ws, const Layout &lo, uint32_t *raw_bits,
                                  int64_t chunk, int64_t *chunk_counts, cudaStream_t st, uint32_t *src_bits = nullptr,
