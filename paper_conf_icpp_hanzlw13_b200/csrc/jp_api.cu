@@ -580,7 +580,21 @@ static jp_status tls_plan(const Job &j, const jp_tls_cfg *cfg, const jp_profile 
       return fail(JP_ERR_ARG, "on-chip TLS recovery needs a profile with waw_iters == 0");
     const int cmax = tls_fwd_max_cluster();
     if (cl > cmax) return fail(JP_ERR_UNSUPPORTED, "the device schedules TLS clusters of up to %d CTAs", cmax);
-    if (path != 0 && path != 5 && path != 6) return fail(JP_ERR_ARG, "on-chip TLS runs on path 5 (cluster) or 6 (grid)");
+    if (path != 0 && path != 5 && path != 6 && path != 8)
+      return fail(JP_ERR_ARG, "on-chip TLS runs on path 5 (cluster), 6 (grid) or 8 (one window)");
+    if (path == 8) {
+      // one window spanning the loop, DC from the guide (jp_tls_flow.cu): ADD_C,
+      // write-once and WAR-free by the profile, guide words of that profile
+      if (j.op != JP_OP_ADD_C || prof->war_iters != 0)
+        return fail(JP_ERR_ARG, "TLS path 8 needs an ADD_C loop whose profile shows war_iters == waw_iters == 0");
+      if (tp.window != 0 && tp.window < j.d.n)
+        return fail(JP_ERR_ARG, "TLS path 8 runs one window of the whole loop (window 0 or >= n)");
+      tp.window = std::max<int64_t>(j.d.n, 1);
+      tp.cluster = num_sms();
+      tp.path = 8;
+      tp.waw = false;
+      return JP_OK;
+    }
     // auto: a window the 16-CTA cluster holds stays there, larger loops use every SM
     if (path == 0) path = (tp.window > 0 ? tp.window : j.d.n) <= tls_fwd_wcap(cmax) ? 5 : 6;
     if (path == 6) {
@@ -752,7 +766,9 @@ static jp_status run_tls_job(const jp_loop *L, const Job &j, const jp_tls_cfg *c
     }
   }
   Layout lo;
-  const int uses = (tp.path == 2 || tp.path == 3 || tp.path == 6 ? JP_WS_TLS : 0) | (tp.guided ? JP_WS_GUIDE : 0);
+  const int uses = (tp.path == 2 || tp.path == 3 || tp.path == 6 || tp.path == 8 ? JP_WS_TLS : 0) |
+                   (tp.guided ? JP_WS_GUIDE : 0);
+  if (tp.path == 8 && !tp.guided) return fail(JP_ERR_ARG, "TLS path 8 needs the guide words (guided = 1)");
   JP_TRY(check_ws(L, ws, ws_bytes, uses, lo));
   if (has_idx(j) && !prof) JP_TRY(validate_sync(j, ws, lo, st, nullptr));
   if (plan_out) *plan_out = tp;
@@ -763,6 +779,10 @@ static jp_status run_tls_job(const jp_loop *L, const Job &j, const jp_tls_cfg *c
     JP_CUDA(launch_serial(j, &hdr[H_TLS_COMMITTED], st), "serial warp");
   } else if (tp.path == 5) {
     JP_CUDA(launch_tls_fwd(j, tp.window, tp.cluster, bits, bsrc, &hdr[H_TLS_COMMITTED], st), "tls on-chip");
+  } else if (tp.path == 8) {
+    auto *V = at<unsigned long long>(ws, lo, R_TLS_C_A);
+    if (!(s_clean & 2)) cudaMemsetAsync(V, 0, 8 * (size_t)L->len_A, st);   // no shadow value yet
+    JP_CUDA(launch_tls_flow(j, bits, bsrc, V, &hdr[H_TLS_COMMITTED], st), "tls one window");
   } else if (tp.path == 6) {
     auto *S = at<unsigned long long>(ws, lo, R_TLS_S_A);
     auto *V = at<unsigned long long>(ws, lo, R_TLS_C_A);
@@ -776,6 +796,12 @@ static jp_status run_tls_job(const jp_loop *L, const Job &j, const jp_tls_cfg *c
   if (stats) {
     int64_t h[4];
     JP_CUDA(d2h_small_sync(h, &hdr[H_TLS_COMMITTED], sizeof h, st), "tls D2H");
+    if (tp.path == 8) {   // device: h[3] violations, h[1] warps that lost their writer
+      if (h[1]) return fail(JP_ERR_ARG, "one-window TLS: a violator's writer never published (guide and profile disagree)");
+      h[0] = L->n;
+      h[1] = L->n + h[3];
+      h[2] = L->n > 0 ? 1 : 0;
+    }
     if (tp.path >= 5 && h[0] < 0)
       return fail(JP_ERR_ARG, "on-chip TLS recovery met an address written twice (the profile passed was wrong)");
     stats->committed = h[0];
@@ -1119,7 +1145,12 @@ static jp_status run_mode(const jp_loop *L, const Job &j, int mode, const jp_pro
     // from the distance-hazard model (restart_plan) unless the caller fixed them
     if (!serial && rec == JP_TLS_RESTART && dist && prof && c.tls_w_max == 0 && c.tls_path == 0 && c.tls_window == 0)
       restart_plan(prof, dist, j.d.n, prof->waw_iters > 0, &wm, &path);
-    jp_tls_cfg tc{c.tls_window, wm, path, 0, 0, rec};
+    // write-once, WAR-free ADD_C loop with the guide already filled by the profile:
+    // one window, DC from the guide, no barrier (path 8, jp_tls_flow.cu)
+    if (rec == JP_TLS_ONCHIP && guide_ready && path == 0 && c.tls_window == 0 && j.op == JP_OP_ADD_C && prof &&
+        prof->war_iters == 0 && prof->waw_iters == 0 && !getenv("JP_TLS_NO_FLOW"))
+      path = 8;
+    jp_tls_cfg tc{c.tls_window, wm, path, 0, path == 8 ? 1 : 0, rec};
     TlsPlan tp;
     JP_TRY(run_tls_job(L, j, &tc, prof, ws, ws_bytes, &res->tls, st, true, &tp, guide_ready, s_clean));
     res->tls_w_max = tp.path == 7 ? 32 : rec == JP_TLS_ONCHIP ? tp.window : wm;

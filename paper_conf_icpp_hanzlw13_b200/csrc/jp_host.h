@@ -59,6 +59,10 @@ bool stamp_pairs_ok(const Job &j, void *ws, const Layout &lo);
 // SAXPY loops over a large A; uses minW/minR_A and maxRx_A as scratch (their
 // tables are NOT left filled).  bucket_profile_ok says whether it applies.
 bool bucket_profile_ok(const Job &j, void *ws, const Layout &lo);
+// one-window on-chip TLS (path 8, jp_tls_flow.cu): ADD_C loops with a profile
+// showing waw = war = 0 and the guide words of that profile; stats as noted there
+cudaError_t launch_tls_flow(const Job &j, const uint32_t *graw, const uint32_t *gsrc, unsigned long long *V,
+                            int64_t *stats, cudaStream_t st);
 cudaError_t launch_prof_bucket(const Job &j, void *ws, const Layout &lo, uint32_t *graw, uint32_t *gsrc,
                                int64_t chunk, int64_t *cc, cudaStream_t st);
 // src_bits (nullable): also the TLS guide's RAW-source words (raw_bits then holds its raw words)

@@ -1,0 +1,180 @@
+// jp_tls_flow.cu -- on-chip TLS recovery (reading B7) with ONE window that spans
+// the whole loop and the dependency check answered by the profile (path 8).
+//
+// Reading B7 (P:L320-333 SE / DC / commit / mis-speculation
+// recovery) runs fixed windows: every iteration speculates against the memory
+// of the window start, DC marks the iterations with an exposed read written by
+// an earlier iteration of the window, the violators are re-executed in
+// dependence order with the operand forwarded from the writer's shadow slot,
+// and the window commits whole.  Its statistics (jpo_sim_tls_fwd) only depend
+// on W.  With W = n the windows -- and the grid barrier between them, ~45% of
+// each window of the all-SM kernel -- disappear:
+//
+//   DC:       the violators of the one window are exactly the raw iterations
+//             (an exposed read written by an earlier iteration of the loop);
+//             the profile's guide (reading B5) already holds that bit, so no
+//             write log is kept and nothing is probed;
+//   SE:       a non-violator's exposed read is of an element no earlier
+//             iteration writes; with write-once (waw = 0) and WAR-free
+//             (war = 0) loops no LATER iteration writes it either, so its value
+//             in A is the window-start value whenever it is read, and the
+//             iteration's result is final: it commits in place at once;
+//   recovery: a violator waits for its writer's shadow slot V[a] = 1 << 32 |
+//             value (published by every RAW source, the guide's second
+//             bitmap), then computes, commits, and publishes in turn.
+//
+// Iterations are dealt in slot sets (i = base + k*G + g) and taken in
+// increasing order by every thread of a co-resident (cooperative) grid: the
+// smallest unfinished iteration only waits for earlier, finished ones, so the
+// sweep cannot deadlock.  Statistics are those of jpo_sim_tls_fwd with W = n:
+// one window, violations = raw iterations, executed = n + violations.
+// ADD_C only (one exposed read of A; configs 1, 3 and the config-5 middle).
+#include <cooperative_groups.h>
+#include "jp_host.h"
+
+namespace cg = cooperative_groups;
+
+namespace jp {
+
+constexpr int kFlowT = 512, kFlowK = 8;
+constexpr unsigned long long kFlowTag = 1ull << 32;
+constexpr long long kFlowSpinLimit = 1ll << 22;   // a lost writer (inconsistent guide) ends the wait with an error
+
+struct FlowSet {
+  int32_t r[kFlowK], w[kFlowK];
+  uint32_t gr[kFlowK], gs[kFlowK];
+  uint32_t x[kFlowK];
+};
+
+template <int DT>
+struct Flow {
+  DLoop L;
+  const uint32_t *graw, *gsrc;
+  unsigned long long *V;
+  uint32_t G, g, n, io;
+  uint32_t viol = 0;
+  bool lost = false;
+
+  __device__ __forceinline__ bool act(uint32_t base, int k) const { return base + (uint32_t)k * G + g < n; }
+  __device__ __forceinline__ uint32_t it(uint32_t base, int k) const { return base + (uint32_t)k * G + g; }
+  __device__ __forceinline__ bool raw_bit(const FlowSet &s, uint32_t base, int k) const {
+    return (s.gr[k] >> (it(base, k) & 31)) & 1u;
+  }
+  __device__ __forceinline__ bool src_bit(const FlowSet &s, uint32_t base, int k) const {
+    return (s.gs[k] >> (it(base, k) & 31)) & 1u;
+  }
+  __device__ __forceinline__ void load(uint32_t base, FlowSet &s) const {
+#pragma unroll
+    for (int k = 0; k < kFlowK; k++) {
+      if (!act(base, k)) continue;
+      const uint32_t i = it(base, k);
+      s.r[k] = L.r ? __ldcs(L.r + i) : (int32_t)(io + i);
+      s.w[k] = L.w ? __ldcs(L.w + i) : (int32_t)(io + i);
+      s.gr[k] = __ldcs(graw + (i >> 5));
+      s.gs[k] = __ldcs(gsrc + (i >> 5));
+    }
+  }
+  // exposed reads of the non-violators (the violators' operands come from V)
+  __device__ __forceinline__ void gather(uint32_t base, FlowSet &s) const {
+#pragma unroll
+    for (int k = 0; k < kFlowK; k++)
+      if (act(base, k) && !raw_bit(s, base, k)) s.x[k] = __ldcg(L.A + s.r[k]);
+  }
+  __device__ __forceinline__ void commit(const FlowSet &s, uint32_t base, int k, uint32_t v) const {
+    __stcg(L.A + s.w[k], v);
+    if (src_bit(s, base, k))
+      asm volatile("st.relaxed.gpu.global.u64 [%0], %1;" ::"l"(V + s.w[k]), "l"(kFlowTag | v) : "memory");
+  }
+  __device__ __forceinline__ void run(uint32_t base, FlowSet &s) {
+    uint32_t pend = 0;
+#pragma unroll
+    for (int k = 0; k < kFlowK; k++) {
+      if (!act(base, k)) continue;
+      if (raw_bit(s, base, k)) pend |= 1u << k;
+      else commit(s, base, k, op_add<DT>(s.x[k], L.c0));
+    }
+    viol += __popc(pend);
+    long long spins = 0;
+    while (__any_sync(0xffffffffu, pend)) {
+#pragma unroll
+      for (int k = 0; k < kFlowK; k++) {
+        if ((pend >> k) & 1u) {
+          unsigned long long v;
+          asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(v) : "l"(V + s.r[k]) : "memory");
+          if ((v >> 32) == 1ull) {
+            commit(s, base, k, op_add<DT>((uint32_t)v, L.c0));
+            pend &= ~(1u << k);
+          }
+        }
+      }
+      if (++spins > kFlowSpinLimit) {   // never on a consistent guide
+        lost = lost || pend;
+        break;
+      }
+    }
+  }
+};
+
+template <int DT>
+__global__ void __launch_bounds__(kFlowT, 1) k_tls_flow(DLoop L, const uint32_t *graw, const uint32_t *gsrc,
+                                                       unsigned long long *V, int64_t *stats) {
+  Flow<DT> F;
+  F.L = L; F.graw = graw; F.gsrc = gsrc; F.V = V;
+  F.G = gridDim.x * (uint32_t)kFlowT;
+  F.g = blockIdx.x * (uint32_t)kFlowT + threadIdx.x;
+  F.n = (uint32_t)L.n;
+  F.io = (uint32_t)L.ioff;
+  const uint32_t step = F.G * (uint32_t)kFlowK;
+  // two slot sets in flight: the next set's indices, guide words and gathers
+  // are issued before this set runs (a non-violator's operand is never written
+  // by another iteration, so it may be read early)
+  FlowSet a, b;
+  F.load(0, a);
+  F.gather(0, a);
+  for (uint32_t base = 0; base < F.n; base += 2 * step) {
+    if (base + step < F.n) { F.load(base + step, b); F.gather(base + step, b); }
+    F.run(base, a);
+    if (base + step >= F.n) break;
+    if (base + 2 * step < F.n) { F.load(base + 2 * step, a); F.gather(base + 2 * step, a); }
+    F.run(base + step, b);
+  }
+  const uint32_t v = __reduce_add_sync(0xffffffffu, F.viol);
+  const unsigned lost = __any_sync(0xffffffffu, F.lost);
+  if ((threadIdx.x & 31) == 0) {
+    if (v) atomicAdd(reinterpret_cast<unsigned long long *>(&stats[3]), (unsigned long long)v);
+    if (lost) atomicAdd(reinterpret_cast<unsigned long long *>(&stats[1]), 1ull);
+  }
+}
+
+template <int DT>
+static cudaError_t run_flow(const Job &j, const uint32_t *graw, const uint32_t *gsrc, unsigned long long *V,
+                            int64_t *stats, cudaStream_t st) {
+  int maxb = 0;
+  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&maxb, (const void *)k_tls_flow<DT>, kFlowT, 0);
+  if (maxb < 1) return cudaErrorInvalidConfiguration;
+  int grid = num_sms();
+  const int64_t need = (j.d.n + kFlowT - 1) / kFlowT;
+  if (need < grid) grid = (int)(need < 1 ? 1 : need);
+  DLoop d = j.d;
+  void *args[] = {&d, &graw, &gsrc, &V, &stats};
+  note_launch();
+  return cudaLaunchCooperativeKernel((const void *)k_tls_flow<DT>, dim3(grid), dim3(kFlowT), args, 0, st);
+}
+
+// Device stats after the kernel: stats[3] = violations (raw iterations),
+// stats[1] = number of warps that gave up waiting for a writer (0 unless the
+// guide was inconsistent); the caller turns them into jpo_sim_tls_fwd's
+// (committed n, executed n + violations, windows 1).  V must hold no value
+// tagged 1 << 32 for an address the loop writes (zeroed).
+cudaError_t launch_tls_flow(const Job &j, const uint32_t *graw, const uint32_t *gsrc, unsigned long long *V,
+                            int64_t *stats, cudaStream_t st) {
+  cudaMemsetAsync(stats, 0, 4 * sizeof(int64_t), st);
+  if (j.d.n == 0) return launch_check();
+  if (j.op != JP_OP_ADD_C) return cudaErrorInvalidValue;
+  cudaError_t e = j.dt == JP_F32 ? run_flow<JP_F32>(j, graw, gsrc, V, stats, st)
+                                 : run_flow<JP_I32>(j, graw, gsrc, V, stats, st);
+  if (e != cudaSuccess) return e;
+  return launch_check();
+}
+
+}  // namespace jp

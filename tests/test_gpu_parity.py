@@ -624,7 +624,7 @@ def test_schedule_stealing_config5(n, chunk, recovery):
     b, e = n // 2, 3 * n // 4   # the TLS task, as a loop of its own
     mid = O.Loop(ref.op, ref.dtype, e - b, ref.A, r=ref.r[b:e], w=ref.w[b:e], c0=ref.c0)
     if recovery == 0:
-        assert res["tls_recovery"] == jp.JP_TLS_ONCHIP and res["tls_path"] in (5, 6) and res["tls_guided"] == 1
+        assert res["tls_recovery"] == jp.JP_TLS_ONCHIP and res["tls_path"] in (5, 6, 8) and res["tls_guided"] == 1
         assert res["tls"] == O.sim_tls_fwd(mid, res["tls_w_max"])[3]
     else:
         assert res["tls_recovery"] == jp.JP_TLS_RESTART and res["tls_path"] == 1

@@ -199,8 +199,9 @@ def test_fwd_config3_full_size_schedule(d):
     L = jp.Loop.from_workload(g)
     res = jp.jp_schedule(L, jp.workspace(L))
     torch.cuda.synchronize()
-    assert res["mode"] == jp.JP_MODE_TLS and res["tls_recovery"] == jp.JP_TLS_ONCHIP and res["tls_path"] == 6
-    assert res["tls_w_max"] == grid_w() and res["tls_guided"] == 1
+    # write-once, WAR-free ADD_C: one window of the whole loop, DC from the guide (path 8)
+    assert res["mode"] == jp.JP_MODE_TLS and res["tls_recovery"] == jp.JP_TLS_ONCHIP and res["tls_path"] == 8
+    assert res["tls_w_max"] == wl.n and res["tls_guided"] == 1
     _, A, _, stats = O.sim_tls_fwd(ref, res["tls_w_max"])
     assert same(g.A, A)
     assert res["tls"] == stats, (res["tls"], stats)
@@ -245,4 +246,95 @@ def test_schedule_fused_guide_bits(case):
     assert np.array_equal(bits_to_flags(words[:nw], wl.n), O.profile(ref)["flags"] & 1)
     assert np.array_equal(bits_to_flags(words[nw:], wl.n), O.raw_sources(ref))
     if res["mode"] == jp.JP_MODE_TLS:
+        assert res["tls"] == O.sim_tls_fwd(ref, res["tls_w_max"])[3]
+
+
+def flow_case(wl, monkey_buckets=None):
+    """jp_run_tls path 8 (one window, DC from the guide) after a profile and the
+    guide on the same workspace: arrays == sequential, stats == jpo_sim_tls_fwd
+    with W = n (one window; violations = raw iterations; executed = n + raw)."""
+    ref = to_oracle(wl)
+    g = wl.to(DEV)
+    L = jp.Loop.from_workload(g)
+    ws = jp.workspace(L)
+    p = jp.jp_profile_density(L, ws)
+    jp.jp_tls_guide(L, ws)
+    got = jp.jp_run_tls(L, window=0, prof=p, ws=ws, guided=True, recovery=jp.JP_TLS_ONCHIP, path=8)
+    torch.cuda.synchronize()
+    st, A, _, stats = O.sim_tls_fwd(ref, max(wl.n, 1))
+    assert same(g.A, A), f"A differs at {np.flatnonzero(g.A.cpu().numpy() != A)[:10]}"
+    assert got == stats, (got, stats)
+    assert got["violations"] == O.profile(ref)["raw_iters"]
+    return got
+
+
+@pytest.mark.parametrize("d", [0.0, 0.001, 0.05, 0.5, 1.0])
+@pytest.mark.parametrize("delta", [1, 64, 1024])
+def test_flow_config3_shapes(d, delta):
+    """Densities up to chains (delta = 1, d = 1: every iteration waits on the previous one)."""
+    n = (1 << 16) + 7 if d < 0.5 or delta > 1 else 5000
+    flow_case(synth.config3(d, n=n, delta=delta))
+
+
+@pytest.mark.parametrize("dt", [O.I32, O.F32])
+@pytest.mark.parametrize("seed", range(3))
+def test_flow_random_write_once(dt, seed):
+    """Write-once ADD_C loops (w a permutation) whose reads are either an earlier
+    iteration's write (RAW) or the iteration's own address -- WAR-free."""
+    g0 = np.random.default_rng(40 + seed)
+    n = [777, 20000, 300001][seed]
+    w = g0.permutation(n).astype(np.int32)
+    r = w.copy()
+    dep = g0.random(n) < 0.3
+    back = np.maximum(np.arange(n) - g0.integers(1, 2000, n), 0)
+    r[dep] = w[back[dep]]
+    A = g0.integers(-1000, 1000, n).astype(np.int32) if dt == O.I32 else g0.standard_normal(n).astype(np.float32)
+    wl = synth.Workload("flow", O.OP_ADD_C, dt, n, torch.from_numpy(A), r=torch.from_numpy(r), w=torch.from_numpy(w),
+                        c0=(3 if dt == O.I32 else 1.1))
+    p = O.profile(to_oracle(wl))
+    assert p["waw_iters"] == 0 and p["war_iters"] == 0
+    flow_case(wl)
+
+
+def test_flow_preconditions():
+    """Path 8 refuses loops it cannot run exactly: WAR present, STENCIL2, no guide."""
+    n = 4000
+    ar = torch.arange(n, dtype=torch.int32)
+    ahead = synth.Workload("ahead", O.OP_ADD_C, O.I32, n, torch.arange(n + 1, dtype=torch.int32), r=ar + 1, w=ar.clone(),
+                           c0=1)     # reads ahead: WAR
+    g = ahead.to(DEV)
+    L = jp.Loop.from_workload(g)
+    ws = jp.workspace(L)
+    p = jp.jp_profile_density(L, ws)
+    assert p["war_iters"] > 0 and p["waw_iters"] == 0
+    jp.jp_tls_guide(L, ws)
+    with pytest.raises(jp.JPError):
+        jp.jp_run_tls(L, prof=p, ws=ws, guided=True, recovery=jp.JP_TLS_ONCHIP, path=8)
+    wl = synth.config3(0.01, n=n)
+    g = wl.to(DEV)
+    L = jp.Loop.from_workload(g)
+    ws = jp.workspace(L)
+    p = jp.jp_profile_density(L, ws)
+    with pytest.raises(jp.JPError):       # no guide words
+        jp.jp_run_tls(L, prof=p, ws=ws, guided=False, recovery=jp.JP_TLS_ONCHIP, path=8)
+    with pytest.raises(jp.JPError):       # a fixed window shorter than the loop
+        jp.jp_tls_guide(L, ws)
+        jp.jp_run_tls(L, window=100, prof=p, ws=ws, guided=True, recovery=jp.JP_TLS_ONCHIP, path=8)
+
+
+def test_schedule_flow_and_windowed_agree(monkeypatch):
+    """jp_schedule picks path 8 for config 3; JP_TLS_NO_FLOW=1 keeps the windowed
+    all-SM kernel (path 6); both reach the sequential state with their own stats."""
+    wl = synth.config3(0.05, n=(1 << 20) + 3)
+    ref = to_oracle(wl)
+    _, A, _ = O.run_seq(ref)
+    for env, path in (("0", 8), ("1", 6)):
+        if env == "1":
+            monkeypatch.setenv("JP_TLS_NO_FLOW", "1")
+        g = wl.to(DEV)
+        L = jp.Loop.from_workload(g)
+        res = jp.jp_schedule(L, jp.workspace(L))
+        torch.cuda.synchronize()
+        assert res["tls_path"] == path, res
+        assert same(g.A, A)
         assert res["tls"] == O.sim_tls_fwd(ref, res["tls_w_max"])[3]
