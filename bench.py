@@ -306,7 +306,7 @@ def crossover_sweep(jp, dev, st, n=1 << 20):
     import synth
     rows = []
     for delta in (1024, 1):
-        for d in (0.10, 0.25, 0.50, 0.75, 1.0):
+        for d in (0.10, 0.25, 0.50, 0.75, 0.90, 0.99, 0.999, 1.0):
             wl = synth.config3(d, n=n, delta=delta, device=dev)
             ref = O.Loop(wl.op, wl.dtype, wl.n, wl.A.cpu().numpy(), r=wl.r.cpu().numpy(), w=wl.w.cpu().numpy(),
                          c0=wl.c0)
@@ -346,7 +346,8 @@ def modes_sweep(jp, dev, st):
     #  profile / guide: jp_profile_density and jp_tls_guide alone
     #  restart_*: the same with restart recovery (reading A6: prefix commit, restart at the first violator)
     tls = []
-    names = {1: "cta", 2: "grid", 3: "cluster16", 4: "tiny", 5: "onchip-cluster", 6: "onchip-grid"}
+    names = {1: "cta", 2: "grid", 3: "cluster16", 4: "tiny", 5: "onchip-cluster", 6: "onchip-grid",
+             7: "serial-warp", 8: "onchip-one-window"}
 
     def timed(fn, A, A0, reps=None):
         """warm up, then the median of `reps` timed runs (20, or

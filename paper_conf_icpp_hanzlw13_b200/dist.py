@@ -276,7 +276,7 @@ def privatized_partitioned(loop, ws, prof, group=None, engine=None, exchange: st
 
 
 def schedule_partitioned(loop, ws, group=None, tau_high: float = 0.25, tls_window: int = 0, tls_w_max: int = 2048,
-                         full_loop=None, engine=None, exchange: str = "dense") -> dict:
+                         full_loop=None, engine=None, exchange: str = "dense", p2p=None) -> dict:
     """Task sharing of one loop across the ranks (P:L342-358 generalised to k
     devices).  ``loop`` is this rank's range (iter_base = its first global id,
     index arrays offset, element arrays shared-address replicas).
@@ -288,7 +288,8 @@ def schedule_partitioned(loop, ws, group=None, tau_high: float = 0.25, tls_windo
         dependence-free special case of PE(V));
         TLS / SEQ_RECOMMENDED: rank 0 runs the windows over ``full_loop`` and
         broadcasts the in/out arrays (replicas only).
-    ``exchange``: "dense" (all_reduce of the tables) or "owner" (NEXT-2).
+    ``exchange``: "dense" (all_reduce of the tables), "owner" (NEXT-2) or "p2p"
+    (small key tables over peer memory; ``p2p`` = handles from ``p2p_handles``).
     """
     jp = _engine(engine)
     world, rank = world_rank(group)
@@ -303,7 +304,7 @@ def schedule_partitioned(loop, ws, group=None, tau_high: float = 0.25, tls_windo
     mode = jp.jp_select_mode(loop, prof, tau_high)
     res = {"mode": mode, "mode_name": _abi.MODE_NAMES[mode], "profiled": 1, "prof": prof, "scheme": "sharing"}
     if mode in (_abi.JP_MODE_DOALL, _abi.JP_MODE_PRIVATIZED):
-        privatized_partitioned(loop, ws, prof, group, jp, exchange)
+        privatized_partitioned(loop, ws, prof, group, jp, exchange, p2p)
     else:
         if full_loop is None:
             raise ValueError("TLS needs the whole loop on rank 0 (full_loop)")

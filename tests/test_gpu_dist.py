@@ -158,17 +158,19 @@ def _p2p_worker(rank, world, port, q):
         loop = full.range(b, e)
         ws = jp.workspace(loop)
         ok = True
-        for _ in range(3):   # epochs 1..3 on the same counter and mappings
+        handles = jd.p2p_handles(loop, ws)   # collective: mapped once, reused by three epochs
+        for ep in range(4):   # epochs 1..3 on the same counter and mappings, then one with handles of its own
             g.T.copy_(T0)
             g.A.copy_(A0)
-            res = jd.schedule_partitioned(loop, ws, full_loop=full, exchange="p2p")
+            res = jd.schedule_partitioned(loop, ws, full_loop=full, exchange="p2p", p2p=handles if ep < 3 else None)
             torch.cuda.synchronize()
             ok &= g.T.cpu().numpy().tobytes() == T_exp.tobytes()
             ok &= g.A.cpu().numpy()[b:e].tobytes() == A_exp[b:e].tobytes()
             ok &= res["mode_name"] == "PRIVATIZED"
-        m = jd._P2P[next(iter(jd._P2P))]
+        m = handles["keys_T"]
         ok &= m.ok() and m.epoch == 3
-        for m in jd._P2P.values():
+        dist.barrier()
+        for m in handles.values():
             m.close()
         q.put((rank, bool(ok)))
     except Exception:  # pragma: no cover
