@@ -542,21 +542,45 @@ def partitioned_config4(jp, dev, st, world, rank, steps):
     prof_ms = timed(lambda: prof.update(jd.profile_partitioned(loop, ws)), steps)
     mode = jp.jp_select_mode(loop, prof, 0.25)
     ms = timed(lambda: jd.privatized_partitioned(loop, ws, prof), steps)
-    ms_p2p = None
-    if world > 1 and IPC_ROWS:
-        handles = jd.p2p_handles(loop, ws)   # collective, once: the IPC mappings outlive the steps
-        ms_p2p = timed(lambda: jd.privatized_partitioned(loop, ws, prof, exchange="p2p", p2p=handles), steps)
-        barrier(world)
-        for h in handles.values():
-            h.close()
     hbm, _ = peaks()
-    return {"workload": "config4: PRIV_TMP fp32 N=2^26 S=1024, task sharing; step = privatized stream + C4 + finalize",
-            "n": wl.n, "n_per_rank": e - b, "mode": jp.MODE_NAMES[mode], "ms": ms, "iters_per_s": wl.n / (ms * 1e-3),
-            "per_rank_frac_of_hbm": BYTES_PER_ITER_PRIV * (e - b) / (ms * 1e-3) / 1e9 / hbm,
-            "profile_ms": prof_ms, "collective": "torch.distributed all_reduce MAX (C4, 8 KiB int64)",
-            "ms_p2p_merge": ms_p2p,
-            "p2p_merge": "C4 as jp_keys_merge_p2p: one CTA per rank reads every rank's 8 KiB over NVLink (CUDA IPC), "
-                         "two device-side barriers, keys applied in the same kernel; no NCCL call"}
+    out = {"workload": "config4: PRIV_TMP fp32 N=2^26 S=1024, task sharing; step = privatized stream + C4 + finalize",
+           "n": wl.n, "n_per_rank": e - b, "mode": jp.MODE_NAMES[mode], "ms": ms, "iters_per_s": wl.n / (ms * 1e-3),
+           "per_rank_frac_of_hbm": BYTES_PER_ITER_PRIV * (e - b) / (ms * 1e-3) / 1e9 / hbm,
+           "profile_ms": prof_ms, "collective": "torch.distributed all_reduce MAX (C4, 8 KiB int64) + finalize"}
+    # C4 over peer memory as a separate single-CTA kernel (jp_keys_merge_p2p)
+    if world > 1 and IPC_ROWS:
+        try:
+            handles = jd.p2p_handles(loop, ws)   # collective, once: the IPC mappings outlive the steps
+            out["ms_p2p_merge"] = timed(lambda: jd.privatized_partitioned(loop, ws, prof, exchange="p2p", p2p=handles),
+                                        steps)
+            barrier(world)
+            for h in handles.values():
+                h.close()
+        except Exception as ex:   # recorded, never fatal to the bench line
+            out["ms_p2p_merge"] = f"error: {ex!r}"[:200]
+    # C4 fused into the stream kernel (jp_priv_stream_merge): one launch per rank and
+    # step, keys pushed into every rank's inbox over NVLink, replayed from a CUDA graph
+    if IPC_ROWS:
+        try:
+            m = jd.PrivMerge(loop, ws)
+            g = m.graph()
+            fn = g.replay if g is not None else m.step
+            fused_ms = timed(fn, steps)
+            m.check()
+            out["fused"] = {"ms": fused_ms, "iters_per_s": wl.n / (fused_ms * 1e-3),
+                            "per_rank_frac_of_hbm": BYTES_PER_ITER_PRIV * (e - b) / (fused_ms * 1e-3) / 1e9 / hbm,
+                            "cuda_graph": g is not None,
+                            "what": "jp_priv_stream_merge: stream + C4 (peer stores + flags) + R2 in one cooperative "
+                                    "kernel per rank; no NCCL call"}
+            if world == 1:   # the merge's fixed cost on one rank: the same stream with its local finalize
+                solo = timed(lambda: jp.jp_run_privatized(loop, prof, ws, stream=st), steps)
+                out["fused"]["stream_alone_ms"] = solo
+                out["fused"]["merge_fixed_cost_us"] = (fused_ms - solo) * 1e3
+            barrier(world)
+            m.close()
+        except Exception as ex:
+            out["fused"] = f"error: {ex!r}"[:200]
+    return out
 
 
 def partitioned_spill(jp, dev, st, world, rank, steps):
@@ -666,20 +690,21 @@ def partitioned_config5(jp, dev, st, world, rank, steps):
     barrier(world)
     ph = jd.schedule_stealing(full, ws, chunk_iters=65536, timings=True)["phases"]
     # device-side stealing (jp_run_priv_claim): chunks claimed at run time
-    dts = []
-    for k in range(4 if world == 1 or IPC_ROWS else 0):
-        wl.A.copy_(A0)
-        torch.cuda.synchronize()
-        barrier(world)
-        t0 = time.perf_counter()
-        dres = jd.schedule_stealing(full, ws, chunk_iters=65536, dynamic=True)
-        torch.cuda.synchronize()
-        barrier(world)
-        if k >= 1:
-            dts.append(time.perf_counter() - t0)
+    dts, dres = [], {"rank_work": "skipped: CUDA-IPC rows turned off (JP_BENCH_IPC=0)"}
+    try:
+        for k in range(4 if world == 1 or IPC_ROWS else 0):
+            wl.A.copy_(A0)
+            torch.cuda.synchronize()
+            barrier(world)
+            t0 = time.perf_counter()
+            dres = jd.schedule_stealing(full, ws, chunk_iters=65536, dynamic=True)
+            torch.cuda.synchronize()
+            barrier(world)
+            if k >= 1:
+                dts.append(time.perf_counter() - t0)
+    except Exception as ex:   # recorded, never fatal to the bench line
+        dts, dres = [], {"rank_work": f"error: {ex!r}"[:200]}
     dyn_ms = max_over_ranks(statistics.median(dts) * 1e3, world, dev) if dts else None
-    if not dts:
-        dres = {"rank_work": "skipped: CUDA-IPC rows at N > 1 need JP_BENCH_IPC=1"}
     phases = {k: max_over_ranks(v, world, dev) for k, v in ph.items()}
     busy = [0.0] * world
     if world > 1:
@@ -750,10 +775,11 @@ def exchange_cost(jp, dev, st):
     return out
 
 
-# Rows that map peer memory through CUDA IPC (spill, p2p C4, device-side
-# stealing) are tested with two ranks sharing one GPU only; on a multi-GPU box
-# they run when JP_BENCH_IPC=1 so that the default scaling run cannot stall on them.
-IPC_ROWS = os.environ.get("JP_BENCH_IPC", "0") == "1"
+# Rows that map peer memory through CUDA IPC (spill, p2p and fused C4, device-side
+# stealing) run at every N (JP_BENCH_IPC=0 turns them off); each is wrapped so an
+# error is recorded in its row instead of ending the run, and every device-side
+# wait has a timeout.
+IPC_ROWS = os.environ.get("JP_BENCH_IPC", "1") == "1"
 
 
 def run_jp(args):
@@ -866,8 +892,11 @@ def run_jp(args):
         torch.cuda.empty_cache()
         part = partitioned_config4(jp, dev, st, world, rank, 5)
         torch.cuda.empty_cache()
-        spill = partitioned_spill(jp, dev, st, world, rank, 5) if world == 1 or IPC_ROWS else \
-            {"skipped": "CUDA-IPC rows at N > 1 need JP_BENCH_IPC=1"}
+        try:
+            spill = partitioned_spill(jp, dev, st, world, rank, 5) if world == 1 or IPC_ROWS else \
+                {"skipped": "CUDA-IPC rows turned off (JP_BENCH_IPC=0)"}
+        except Exception as ex:   # recorded, never fatal to the bench line
+            spill = {"error": repr(ex)[:200]}
         torch.cuda.empty_cache()
         steal = partitioned_config5(jp, dev, st, world, rank, 10)
         torch.cuda.empty_cache()

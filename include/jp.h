@@ -497,6 +497,26 @@ jp_status jp_run_doall_spill(const jp_loop *views /* host [world] */, int32_t wo
 jp_status jp_keys_merge_p2p(const int64_t *const *peer_keys /* host [world] */, int32_t world, int64_t *keys,
                             int64_t len, unsigned long long *bar, int64_t epoch, void *arr, int32_t *err,
                             jp_stream_t st);
+/* Privatized stream + C4 + R2 in ONE kernel per rank (config-4 shape: PRIV_TMP,
+ * identity X / Y, indirect s, len_T <= 4096; SURVEY Sec.8(e) "C4 ... or inside
+ * the kernel"; the paper updates privatized variables "after all the iterations
+ * finish execution", reading A9).  L is this rank's range
+ * (iter_base = global id of its first iteration).  After every CTA's key flush
+ * and a grid barrier, one CTA pushes this rank's len_T packed keys into slot
+ * (epoch parity, me) of EVERY rank's inbox (plain stores to peer memory over
+ * NVLink), raises one release flag per peer, waits for all world flags of this
+ * epoch in its own inbox, reduces the world tables (MAX, local loads) and
+ * applies the last writers to T.  inbox: jp_priv_inbox_bytes bytes per rank,
+ * zeroed once before the first call; peer_inbox (host [world]) holds every
+ * rank's inbox pointer as mapped in this process (own included; CUDA IPC).
+ * The epoch lives in the inbox, so the call's launches (a key memset and one
+ * cooperative kernel) take the same arguments every step: a CUDA graph can
+ * capture them.  Every rank calls it once per step; a wait over ~4 s sets *err
+ * (device int32, caller zeroes) to 1 and leaves T unmerged.  Stream-ordered.   */
+size_t jp_priv_inbox_bytes(const jp_loop *L /* host */, int32_t world);
+jp_status jp_priv_stream_merge(const jp_loop *L, const jp_profile *p /* host, nullable */, void *ws, size_t ws_bytes,
+                               void *const *peer_inbox /* host [world] */, int32_t world, int32_t me,
+                               int32_t *err, jp_stream_t st);
 /* CUDA IPC plumbing for the spill (peer shards and the counter table):
  * export: a 64-byte handle (host) of the allocation holding ptr, and ptr's
  * byte offset in it; import (in another process): *ptr = mapped base + offset

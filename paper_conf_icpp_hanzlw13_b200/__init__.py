@@ -26,7 +26,7 @@ __all__ = [
     "jp_profile_classify", "jp_profile_density", "jp_select_mode", "jp_run_doall", "jp_run_privatized",
     "jp_priv_stream", "jp_priv_finalize", "jp_doall_kernel", "jp_tls_guide", "jp_tls_next_window", "jp_run_tls", "jp_schedule", "jp_stage_bytes", "jp_schedule_host",
     "jp_plan_sharing", "jp_plan_stealing", "jp_merge_apply",
-    "jp_plan", "jp_plan_tasks", "jp_export_keys", "jp_keys_merge_p2p", "jp_run_priv_claim", "jp_run_doall_spill", "jp_ipc_export", "jp_ipc_import", "jp_ipc_close",
+    "jp_plan", "jp_plan_tasks", "jp_export_keys", "jp_keys_merge_p2p", "jp_priv_inbox_bytes", "jp_priv_stream_merge", "jp_run_priv_claim", "jp_run_doall_spill", "jp_ipc_export", "jp_ipc_import", "jp_ipc_close",
     "jp_sparse_scratch_bytes", "jp_sparse_pack", "jp_sparse_reduce_max", "jp_sparse_gather", "jp_sparse_scatter",
     "jp_last_error", "jp_version", "jp_launch_count", "jp_tls_grid_window",
 ]
@@ -411,6 +411,18 @@ def jp_keys_merge_p2p(peer_ptrs, keys: torch.Tensor, bar, epoch: int, err: torch
     pp = (C.c_void_p * len(peer_ptrs))(*[int(p) for p in peer_ptrs])
     check(lib().jp_keys_merge_p2p(pp, len(peer_ptrs), keys.data_ptr(), keys.numel(), bar.data_ptr(), int(epoch),
                                   _ptr(arr), err.data_ptr(), _stream(stream)))
+
+
+def jp_priv_inbox_bytes(loop: Loop, world: int) -> int:
+    return int(lib().jp_priv_inbox_bytes(loop.ref, int(world)))
+
+
+def jp_priv_stream_merge(loop: Loop, ws, inbox_ptrs, me: int, err: torch.Tensor, prof=None, stream=None):
+    """inbox_ptrs: every rank's inbox pointer as mapped here (ints, own included)."""
+    pp = (C.c_void_p * len(inbox_ptrs))(*[int(p) for p in inbox_ptrs])
+    p, nb = _ws(ws)
+    check(lib().jp_priv_stream_merge(loop.ref, _pref(prof), p, nb, pp, len(inbox_ptrs), int(me), err.data_ptr(),
+                                     _stream(stream)))
 
 
 def jp_ipc_export(t: torch.Tensor) -> tuple[bytes, int]:

@@ -117,6 +117,8 @@ SIGNATURES = [
     ("jp_export_keys", _I32, [_P(jp_loop), _V, _SZ, _V]),
     ("jp_run_priv_claim", _I32, [_P(jp_loop), _V, _P(_I64), _I32, _I32, _V, _V, _V, _SZ, _I32, _V]),
     ("jp_keys_merge_p2p", _I32, [_P(_V), _I32, _V, _I64, _V, _I64, _V, _V, _V]),
+    ("jp_priv_inbox_bytes", _SZ, [_P(jp_loop), _I32]),
+    ("jp_priv_stream_merge", _I32, [_P(jp_loop), _P(jp_profile), _V, _SZ, _P(_V), _I32, _I32, _V, _V]),
     ("jp_run_doall_spill", _I32, [_P(jp_loop), _I32, _I32, _I64, _V, _V, _I32, _V]),
     ("jp_ipc_export", _I32, [_V, _V, _P(_I64)]),
     ("jp_ipc_import", _I32, [_V, _I64, _P(_V)]),

@@ -889,6 +889,33 @@ jp_status jp_keys_merge_p2p(const int64_t *const *peer_keys, int32_t world, int6
   return JP_OK;
 }
 
+size_t jp_priv_inbox_bytes(const jp_loop *L, int32_t world) {
+  if (check_loop(L) != JP_OK) return 0;
+  return priv_inbox_bytes(make_job(L), world);
+}
+
+jp_status jp_priv_stream_merge(const jp_loop *L, const jp_profile *p, void *ws, size_t ws_bytes,
+                               void *const *peer_inbox, int32_t world, int32_t me, int32_t *err, jp_stream_t st) {
+  JP_TRY(check_loop(L));
+  if (p && p->raw_iters != 0) return fail(JP_ERR_ILLEGAL_MODE, "privatization needs d_raw = 0");
+  const Job j = make_job(L);
+  if (!priv_merge_ok(j, world))
+    return fail(JP_ERR_UNSUPPORTED, "the fused merge runs PRIV_TMP with identity X / Y, an indirect s, "
+                                    "len_T <= 4096, 16-byte aligned streams and 1 <= world <= 8");
+  if (!peer_inbox || me < 0 || me >= world || !err) return fail(JP_ERR_ARG, "bad merge arguments");
+  for (int k = 0; k < world; k++)
+    if (!peer_inbox[k]) return fail(JP_ERR_ARG, "inbox of rank %d is NULL", k);
+  JP_TRY(need_device());
+  Layout lo;
+  JP_TRY(check_ws(L, ws, ws_bytes, JP_WS_PRIV, lo));
+  if (L->n == 0) return JP_OK;
+  JP_CUDA(launch_priv_stream_merge(j, at<unsigned long long>(ws, lo, R_KEYS_T),
+                                   reinterpret_cast<unsigned long long *const *>(peer_inbox), world, me, err,
+                                   (cudaStream_t)st),
+          "priv stream + merge");
+  return JP_OK;
+}
+
 typedef int (*cu_range_fn)(unsigned long long *, size_t *, unsigned long long);
 static cu_range_fn cu_mem_range() {
   static cu_range_fn fn = nullptr;

@@ -91,6 +91,12 @@ cudaError_t launch_serial(const Job &j, int64_t *stats, cudaStream_t st);
 cudaError_t launch_priv_claim(const Job &j, void *ws, const Layout &lo, const int64_t *chunks, const int64_t *first,
                               int world, int me, unsigned long long *ctr, int64_t *stats, int max_ctas,
                               cudaStream_t st);
+// the privatized stream of a config-4-shaped rank range with C4 over peer memory and
+// R2 fused into its epilogue (jp_priv_stream_merge); inbox = every rank's inbox mapped here
+bool priv_merge_ok(const Job &j, int world);
+size_t priv_inbox_bytes(const Job &j, int world);
+cudaError_t launch_priv_stream_merge(const Job &j, unsigned long long *kT, unsigned long long *const *inbox, int world,
+                                     int me, int *err, cudaStream_t st);
 // C4 over NVLink peer memory: merged max of every rank's key table (len <= kP2PMaxLen), applied to arr
 constexpr int64_t kP2PMaxLen = 16384;
 cudaError_t launch_keys_merge_p2p(const unsigned long long *const *peers, int world, unsigned long long *mine,

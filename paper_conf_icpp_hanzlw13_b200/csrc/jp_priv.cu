@@ -155,9 +155,81 @@ constexpr int kPrivTile = 4096, kPrivStages = 4, kPrivTmaThreads = 256;
 // grid-wide barrier, then the merged keys are applied to T in the same kernel
 // (R1 + R2 in one launch, single-GPU jp_run_privatized only: across GPUs the
 // keys are merged by C4 between the stream and the finalize).
-template <int DT>
+// C4 fused into the stream (jp_priv_stream_merge): every rank's inbox holds
+//   [0] epoch of the last merge, [32 + 2*8] flags[parity][sender] = epoch,
+//   [64 ...] keys[parity][sender][lenT]
+// and every rank maps every rank's inbox (CUDA IPC / NVLink peer memory).
+constexpr int kMergePeers = 8;
+constexpr int64_t kInboxFlags = 32, kInboxKeys = 64;
+struct MergeP2P {
+  unsigned long long *inbox[kMergePeers];   // every rank's inbox, mapped here (own included)
+  int world, me;
+  int *err;
+};
+
+__device__ __forceinline__ unsigned long long gtimer_ns() {
+  unsigned long long t;
+  asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
+  return t;
+}
+
+// One CTA, after the grid barrier that follows every CTA's key flush: push this
+// rank's keys into slot (parity, me) of every rank's inbox with plain peer
+// stores (posted over NVLink), a system fence, then one release flag per peer;
+// wait for every sender's flag of this epoch in the local inbox; reduce the
+// world key tables (local loads) and apply the merged last writers to T.
+// Double-buffered by epoch parity: a rank writes parity e+1 only after its
+// merge e, which needed every peer's flag e, i.e. every peer's push e -- pushes
+// of e+1 never land in a buffer a peer still reduces for e-1.
+__device__ void merge_p2p_epilogue(const DLoop &L, const unsigned long long *kT, const MergeP2P &M) {
+  __shared__ unsigned long long e_s;
+  __shared__ int ok;
+  unsigned long long *in = M.inbox[M.me];
+  const int tid = threadIdx.x, nt = blockDim.x;
+  const int64_t lenT = L.lenT;
+  if (tid == 0) { e_s = in[0] + 1; ok = 1; }
+  __syncthreads();
+  const unsigned long long e = e_s;
+  const int par = (int)(e & 1);
+  for (int p = 0; p < M.world; p++) {
+    unsigned long long *dst = M.inbox[p] + kInboxKeys + ((int64_t)par * M.world + M.me) * lenT;
+    for (int64_t b = tid; b < lenT; b += nt) dst[b] = __ldcg(kT + b);
+  }
+  __threadfence_system();
+  __syncthreads();
+  if (tid < M.world) {
+    unsigned long long *f = M.inbox[tid] + kInboxFlags + par * kMergePeers + M.me;
+    asm volatile("st.release.sys.global.u64 [%0], %1;" ::"l"(f), "l"(e) : "memory");
+    // ... and wait for sender tid's flag of this epoch here
+    const unsigned long long *g = in + kInboxFlags + par * kMergePeers + tid;
+    const unsigned long long t0 = gtimer_ns();
+    for (;;) {
+      unsigned long long v;
+      asm volatile("ld.acquire.sys.global.u64 %0, [%1];" : "=l"(v) : "l"(g) : "memory");
+      if (v >= e) break;
+      if (gtimer_ns() - t0 > 4000000000ull) { ok = 0; atomicExch(M.err, 1); break; }
+      __nanosleep(100);
+    }
+  }
+  __syncthreads();
+  if (!ok) return;
+  asm volatile("fence.acq_rel.sys;" ::: "memory");
+  const unsigned long long *keys = in + kInboxKeys + (int64_t)par * M.world * lenT;
+  for (int64_t b = tid; b < lenT; b += nt) {
+    unsigned long long m = 0;
+    for (int r = 0; r < M.world; r++) {
+      const unsigned long long v = __ldcv(keys + (int64_t)r * lenT + b);
+      m = v > m ? v : m;
+    }
+    if (m) L.T[b] = (uint32_t)m;
+  }
+  __syncthreads();
+  if (tid == 0) in[0] = e;
+}
+
+template <int DT, bool MERGE = false>
 __global__ void __launch_bounds__(kPrivTmaThreads, 1) k_priv_tmp_tma(DLoop L, unsigned long long *kT, int64_t ntiles,
-                                                                     int fuse_apply) {
+                                                                     int fuse_apply, MergeP2P M = MergeP2P{}) {
   if (aborted(L)) return;
   extern __shared__ __align__(128) uint32_t psm[];   // [stage][2][tile] then tT[lenT]
   __shared__ __align__(8) unsigned long long full[kPrivStages];
@@ -231,6 +303,10 @@ __global__ void __launch_bounds__(kPrivTmaThreads, 1) k_priv_tmp_tma(DLoop L, un
   }
   if (fuse_apply) {
     cg::this_grid().sync();   // every CTA's keys are in
+    if constexpr (MERGE) {   // C4 across the ranks, then R2, in CTA 0
+      if (blockIdx.x == 0) merge_p2p_epilogue(L, kT, M);
+      return;
+    }
     for (int64_t b = (int64_t)blockIdx.x * kPrivTmaThreads + tid; b < L.lenT; b += (int64_t)gridDim.x * kPrivTmaThreads) {
       const unsigned long long k = __ldcg(&kT[b]);
       if (k) L.T[b] = (uint32_t)k;
@@ -275,7 +351,7 @@ static void run_priv(const DLoop &d0, unsigned long long *kA, unsigned long long
       if (doall_kernel_choice() == 1) {   // bulk-copy staged (the DOALL kernel choice covers both streams)
         const int64_t ntiles = d.n / kPrivTile;
         const size_t smem = (size_t)kPrivStages * 2 * kPrivTile * 4 + (size_t)d.lenT * 4;
-        cudaFuncSetAttribute(k_priv_tmp_tma<DT>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+        cudaFuncSetAttribute(k_priv_tmp_tma<DT, false>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
         int g = num_sms();
         if (max_ctas > 0 && g > max_ctas) g = max_ctas;
         if (ntiles < g) g = (int)(ntiles < 1 ? 1 : ntiles);
@@ -284,12 +360,13 @@ static void run_priv(const DLoop &d0, unsigned long long *kA, unsigned long long
           DLoop dd = d;
           int64_t nt = ntiles;
           validate_first();
-          void *args[] = {&dd, &kT, &nt, &fuse};
-          cudaLaunchCooperativeKernel((void *)k_priv_tmp_tma<DT>, dim3(g), dim3(kPrivTmaThreads), args, smem, st);
+          MergeP2P none{};
+          void *args[] = {&dd, &kT, &nt, &fuse, &none};
+          cudaLaunchCooperativeKernel((void *)k_priv_tmp_tma<DT, false>, dim3(g), dim3(kPrivTmaThreads), args, smem, st);
           *applied = true;
         } else {
           validate_first();
-          k_priv_tmp_tma<DT><<<g, kPrivTmaThreads, smem, st>>>(d, kT, ntiles, 0);
+          k_priv_tmp_tma<DT, false><<<g, kPrivTmaThreads, smem, st>>>(d, kT, ntiles, 0, MergeP2P{});
         }
         note_launch();
         return;
@@ -311,6 +388,47 @@ static void run_priv(const DLoop &d0, unsigned long long *kA, unsigned long long
   validate_first();
   k_priv_generic<OP, DT><<<grid, kPrivThreads, smem, st>>>(d, kA, kT, smA, smT);
   note_launch();
+}
+
+bool priv_merge_ok(const Job &j, int world) {
+  const DLoop &d = j.d;
+  return j.op == JP_OP_PRIV_TMP && !d.r && !d.w && d.s && d.lenT > 0 && d.lenT <= kSmemSlots && world >= 1 &&
+         world <= kMergePeers && al16(d.X + d.ioff) && al16(d.s) && al16(d.A + d.ioff);
+}
+
+size_t priv_inbox_bytes(const Job &j, int world) {
+  return priv_merge_ok(j, world) ? 8 * ((size_t)kInboxKeys + 2 * (size_t)world * (size_t)j.d.lenT) : 0;
+}
+
+cudaError_t launch_priv_stream_merge(const Job &j, unsigned long long *kT, unsigned long long *const *inbox, int world,
+                                     int me, int *err, cudaStream_t st) {
+  DLoop d = j.d;   // rank-local range (B1): X and Y rebased to the range's first element
+  d.X += d.ioff; d.lenX -= d.ioff;
+  d.A += d.ioff; d.lenA -= d.ioff;
+  d.ioff = 0;
+  cudaMemsetAsync(kT, 0, 8 * (size_t)d.lenT, st);
+  const int64_t ntiles = d.n / kPrivTile;
+  const size_t smem = (size_t)kPrivStages * 2 * kPrivTile * 4 + (size_t)d.lenT * 4;
+  cudaError_t e;
+  auto go = [&](auto kern) {
+    cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+    int g = num_sms();
+    if (ntiles < g) g = (int)(ntiles < 1 ? 1 : ntiles);
+    MergeP2P M{};
+    for (int k = 0; k < world; k++) M.inbox[k] = inbox[k];
+    M.world = world;
+    M.me = me;
+    M.err = err;
+    int fuse = 1;
+    int64_t nt = ntiles;
+    void *args[] = {&d, &kT, &nt, &fuse, &M};
+    e = cudaLaunchCooperativeKernel((const void *)kern, dim3(g), dim3(kPrivTmaThreads), args, smem, st);
+  };
+  if (j.dt == JP_F32) go(k_priv_tmp_tma<JP_F32, true>);
+  else go(k_priv_tmp_tma<JP_I32, true>);
+  note_launch();
+  if (e != cudaSuccess) return e;
+  return launch_check();
 }
 
 cudaError_t launch_priv_stream(const Job &j, void *ws, const Layout &lo, bool clear_keys, cudaStream_t st,

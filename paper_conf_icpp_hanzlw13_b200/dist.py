@@ -180,6 +180,69 @@ class P2PMerge:
         self._opened = []
 
 
+class PrivMerge:
+    """Config 4 across the ranks in ONE kernel per rank and step
+    (jp_priv_stream_merge): privatized stream of this rank's range, C4 by peer
+    stores into every rank's inbox (CUDA IPC / NVLink), R2 -- no NCCL call, no
+    second launch.  Collective to build (every rank maps every rank's inbox
+    once); ``step()`` launches, ``check()`` synchronizes and raises if a merge
+    timed out; ``graph()`` captures one step in a CUDA graph (same arguments
+    every step: the epoch lives in the inbox) and returns a replay callable."""
+
+    def __init__(self, loop, ws, group=None, engine=None):
+        jp = _engine(engine)
+        self.jp, self.loop, self.ws, self.group = jp, loop, ws, group
+        self.world, self.rank = world_rank(group)
+        nb = jp.jp_priv_inbox_bytes(loop, self.world)
+        if nb == 0:
+            raise ValueError("the fused merge needs the config-4 shape (PRIV_TMP, identity X/Y, indirect s, "
+                             "len_T <= 4096)")
+        dev = ws.device
+        self.inbox = torch.zeros(nb // 8, dtype=torch.int64, device=dev)
+        self.err = torch.zeros(1, dtype=torch.int32, device=dev)
+        self._opened = []
+        torch.cuda.synchronize()
+        if self.world == 1:
+            self.ptrs = [self.inbox.data_ptr()]
+        else:
+            allinfo = [None] * self.world
+            dist.all_gather_object(allinfo, jp.jp_ipc_export(self.inbox), group=group)
+            self.ptrs = []
+            for k, h in enumerate(allinfo):
+                if k == self.rank:
+                    self.ptrs.append(self.inbox.data_ptr())
+                else:
+                    p = jp.jp_ipc_import(*h)
+                    self._opened.append((p, h[1]))
+                    self.ptrs.append(p)
+            dist.barrier(group=group)
+
+    def step(self, stream=None):
+        self.jp.jp_priv_stream_merge(self.loop, self.ws, self.ptrs, self.rank, self.err, stream=stream)
+
+    def check(self):
+        torch.cuda.synchronize()
+        if int(self.err.item()) != 0:
+            raise RuntimeError(f"fused privatized merge: a peer's flag never arrived on rank {self.rank}")
+
+    def graph(self):
+        """One step captured in a CUDA graph (replayed with g.replay()); None if
+        the driver refuses to capture the cooperative launch."""
+        try:
+            s = torch.cuda.Stream()
+            g = torch.cuda.CUDAGraph()
+            with torch.cuda.graph(g, stream=s):
+                self.step()
+            return g
+        except Exception:   # pragma: no cover - capture support is driver-dependent
+            return None
+
+    def close(self):
+        for p, off in self._opened:
+            self.jp.jp_ipc_close(p, off)
+        self._opened = []
+
+
 def p2p_handles(loop, ws, group=None, engine=None) -> dict:
     """Collective: one P2PMerge per small key table of ``loop`` in ``ws`` (every
     rank must call it with its own replica).  The handles keep the tables (and
