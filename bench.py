@@ -540,7 +540,7 @@ def partitioned_config4(jp, dev, st, world, rank, steps):
 
     prof = {}
     prof_ms = timed(lambda: prof.update(jd.profile_partitioned(loop, ws)), steps)
-    mode = jp.jp_select_mode(loop, prof, 0.25)
+    mode = jp.jp_select_mode(loop, prof)
     ms = timed(lambda: jd.privatized_partitioned(loop, ws, prof), steps)
     hbm, _ = peaks()
     out = {"workload": "config4: PRIV_TMP fp32 N=2^26 S=1024, task sharing; step = privatized stream + C4 + finalize",

@@ -137,7 +137,7 @@ typedef struct {
 typedef struct {
   int32_t scheme;               /* jp_scheme                                          */
   int32_t tls_path;             /* jp_tls_cfg.path                                    */
-  double tau_high;              /* Fig. 2(b) "(Density > N)" threshold, reading A4 (0.25) */
+  double tau_high;              /* Fig. 2(b) "(Density > N)" threshold, reading A4 (0.999, measured) */
   int64_t chunk_iters;          /* task size for stealing / sharing (reading A17)     */
   int64_t tls_window;           /* jp_tls_cfg.window                                  */
   int64_t tls_w_max;            /* jp_tls_cfg.w_max; 0 = auto from the profiled

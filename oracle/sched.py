@@ -9,7 +9,7 @@ import math
 DOALL, PRIVATIZED, TLS, SEQ_RECOMMENDED = 0, 1, 2, 3
 
 
-def select_mode(all_null: bool, n: int, raw: int, war: int, waw: int, tau_high: float = 0.25) -> int:
+def select_mode(all_null: bool, n: int, raw: int, war: int, waw: int, tau_high: float = 0.999) -> int:
     """Fig. 2(b) workflow, readings A4 and A5:
     determined DOALL? -> A;  TD density high -> C;  low -> B;  FD -> D;  else D'."""
     if all_null:

@@ -178,7 +178,7 @@ def jp_profile_density(loop: Loop, ws, raw_bits=None, chunk_iters=0, chunk_count
     return _prof_dict(out)
 
 
-def jp_select_mode(loop: Loop, prof=None, tau_high: float = 0.25) -> int:
+def jp_select_mode(loop: Loop, prof=None, tau_high: float = _abi.TAU_HIGH) -> int:
     m = lib().jp_select_mode(loop.ref, _pref(prof), float(tau_high))
     if m < 0:
         raise JPError(_abi.JP_ERR_ARG, lib().jp_last_error().decode())
@@ -246,7 +246,7 @@ def jp_run_tls(loop: Loop, window=0, w_max=65536, path=0, prof=None, ws=None, st
     return {k: getattr(st, k) for k, _ in _abi.jp_tls_stats._fields_} if stats else None
 
 
-def sched_cfg(scheme=JP_SCHED_SHARING, tau_high=0.25, chunk_iters=65536, tls_window=0, tls_w_max=0,
+def sched_cfg(scheme=JP_SCHED_SHARING, tau_high=_abi.TAU_HIGH, chunk_iters=65536, tls_window=0, tls_w_max=0,
               tls_path=0, tls_recovery=0, static_check=0) -> _abi.jp_sched_cfg:
     """tls_recovery: 0 auto (on chip when the profile shows waw_iters == 0), 1 restart, 2 on chip.
     static_check: 0 run jp_static_check before profiling, 1 skip it."""
@@ -366,7 +366,7 @@ def jp_plan(loop: Loop, chunk_profiles, world: int, speed=None, cfg=None, **kw):
     return [tuple(out[4 * k:4 * k + 4]) for k in range(n.value)]
 
 
-def jp_plan_tasks(loop: Loop, chunk_counts, chunk_iters: int, ws, tau_high: float = 0.25, stream=None):
+def jp_plan_tasks(loop: Loop, chunk_counts, chunk_iters: int, ws, tau_high: float = _abi.TAU_HIGH, stream=None):
     """chunk_counts: the whole loop's (raw, war, waw) per chunk (flat list / int64
     tensor).  Returns ([(start, end, mode)], conf list of 64 ints)."""
     cc = [int(x) for x in (chunk_counts.tolist() if hasattr(chunk_counts, "tolist") else chunk_counts)]

@@ -134,6 +134,9 @@ SIGNATURES = [
     ("jp_tls_grid_window", _I64, []),
 ]
 
+# reading A4's Fig. 2(b) threshold, the library's default (jp_host.h kTauHigh, measured)
+TAU_HIGH = 0.999
+
 _lock = threading.Lock()
 _lib = None
 

@@ -1123,7 +1123,7 @@ static jp_sched_cfg default_cfg() {
   jp_sched_cfg c;
   memset(&c, 0, sizeof c);
   c.scheme = JP_SCHED_SHARING;
-  c.tau_high = 0.25;
+  c.tau_high = kTauHigh;
   c.chunk_iters = 65536;
   c.tls_window = 0;
   c.tls_w_max = 0;   // auto from the profiled density (auto_w_max)
@@ -1498,7 +1498,7 @@ jp_status jp_plan(const jp_loop *L, const jp_sched_cfg *cfg, const jp_profile *c
     hc[3 * k + 1] = chunk_profiles[k].war_iters;
     hc[3 * k + 2] = chunk_profiles[k].waw_iters;
   }
-  std::vector<Task> tk = chunk_tasks(hc.data(), L->n, chunk, cfg->tau_high > 0.0 ? cfg->tau_high : 0.25);
+  std::vector<Task> tk = chunk_tasks(hc.data(), L->n, chunk, cfg->tau_high > 0.0 ? cfg->tau_high : kTauHigh);
   std::vector<int64_t> tasks;
   for (const Task &t : tk) { tasks.push_back(t.s); tasks.push_back(t.e); tasks.push_back(t.mode); }
   if (cfg->scheme == JP_SCHED_STEALING)
@@ -1533,7 +1533,7 @@ jp_status jp_plan_tasks(const jp_loop *L, const int64_t *chunk_counts, int64_t c
   JP_TRY(need_device());
   Layout lo;
   JP_TRY(check_ws(L, ws, ws_bytes, JP_WS_ALL, lo));
-  std::vector<Task> tk = chunk_tasks(chunk_counts, L->n, chunk_iters, tau_high > 0.0 ? tau_high : 0.25);
+  std::vector<Task> tk = chunk_tasks(chunk_counts, L->n, chunk_iters, tau_high > 0.0 ? tau_high : kTauHigh);
   std::vector<unsigned long long> cf;
   JP_TRY(task_conflicts(make_job(L), L, ws, lo, tk, chunk_iters, cf, (cudaStream_t)st));
   *n_tasks = (int32_t)tk.size();
@@ -1572,7 +1572,7 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
   if (!res) return fail(JP_ERR_ARG, "result is NULL");
   JP_TRY(need_device());
   jp_sched_cfg c = cfgp ? *cfgp : default_cfg();
-  if (c.tau_high <= 0.0) c.tau_high = 0.25;
+  if (c.tau_high <= 0.0) c.tau_high = kTauHigh;
   if (c.chunk_iters <= 0) c.chunk_iters = 65536;
   if (c.tls_w_max < 0) c.tls_w_max = 0;
   memset(res, 0, sizeof *res);

@@ -24,6 +24,12 @@ Layout layout(const jp_loop *L);
 // End of the furthest region the JP_WS_* uses touch.
 size_t layout_end(const Layout &lo, int uses);
 constexpr int64_t kSchedMinChunk = 1024;
+// Reading A4's threshold of Fig. 2(b) "(Density > N)", measured: the
+// one-window on-chip TLS beats the one-warp program-order path (mode C) on every
+// loop of the crossover sweep up to d_raw = 0.999 (chains, delta = 1: 131 vs 19 M
+// committed iter/s at 0.999; 0.88 vs 18.95 at 1.0), so mode C starts above 0.999
+// (bench.py modes.crossover, profiles/r02_bench.json; DESIGN.md Sec.3 A4)
+constexpr double kTauHigh = 0.999;
 constexpr int kMaxTasks = 64;
 // scheduler scratch sub-layout (inside R_SCHED)
 struct SchedLayout {

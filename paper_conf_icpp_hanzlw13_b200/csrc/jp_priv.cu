@@ -195,7 +195,8 @@ __device__ void merge_p2p_epilogue(const DLoop &L, const unsigned long long *kT,
     unsigned long long *dst = M.inbox[p] + kInboxKeys + ((int64_t)par * M.world + M.me) * lenT;
     for (int64_t b = tid; b < lenT; b += nt) dst[b] = __ldcg(kT + b);
   }
-  __threadfence_system();
+  // the CTA barrier orders every thread's pushes before the flag writers'
+  // system-scope release (cumulative): no fence per pushing thread
   __syncthreads();
   if (tid < M.world) {
     unsigned long long *f = M.inbox[tid] + kInboxFlags + par * kMergePeers + M.me;

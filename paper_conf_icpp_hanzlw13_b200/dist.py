@@ -338,7 +338,7 @@ def privatized_partitioned(loop, ws, prof, group=None, engine=None, exchange: st
         jp.jp_priv_finalize(loop, ws)
 
 
-def schedule_partitioned(loop, ws, group=None, tau_high: float = 0.25, tls_window: int = 0, tls_w_max: int = 2048,
+def schedule_partitioned(loop, ws, group=None, tau_high: float = _abi.TAU_HIGH, tls_window: int = 0, tls_w_max: int = 2048,
                          full_loop=None, engine=None, exchange: str = "dense", p2p=None) -> dict:
     """Task sharing of one loop across the ranks (P:L342-358 generalised to k
     devices).  ``loop`` is this rank's range (iter_base = its first global id,
@@ -391,7 +391,7 @@ def _levels(conf, nt):
     return lv
 
 
-def schedule_stealing(full, ws, group=None, chunk_iters: int = 65536, tau_high: float = 0.25, speed=None,
+def schedule_stealing(full, ws, group=None, chunk_iters: int = 65536, tau_high: float = _abi.TAU_HIGH, speed=None,
                       speed_tls: float = 1.0, exchange: str = "dense", engine=None, timings: bool = False,
                       dynamic: bool = False) -> dict:
     """Task stealing of one loop across the ranks (Alg. 1; SURVEY

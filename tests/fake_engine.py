@@ -241,7 +241,7 @@ def jp_sparse_scatter(t0, t1, rows):
 
 
 # ---- task stealing across ranks (jp.h jp_plan_tasks / jp_export_keys), plain definitions ----
-def jp_plan_tasks(loop, chunk_counts, chunk_iters, ws, tau_high=0.25):
+def jp_plan_tasks(loop, chunk_counts, chunk_iters, ws, tau_high=0.999):
     import oracle.sched as OS
     cc = [int(x) for x in (chunk_counts.tolist() if hasattr(chunk_counts, "tolist") else chunk_counts)]
     n = loop.n

@@ -97,7 +97,8 @@ def test_select_mode_paper_cases():
                              "d_raw": r / n, "d_war": a / n, "d_waw": b / n}
     assert jp.jp_select_mode(L, mk(1000, 12, 0, 0)) == jp.JP_MODE_TLS
     assert jp.jp_select_mode(L, mk(1000, 0, 900, 900)) == jp.JP_MODE_PRIVATIZED
-    assert jp.jp_select_mode(L, mk(1000, 999, 999, 0)) == jp.JP_MODE_SEQ_RECOMMENDED
+    assert jp.jp_select_mode(L, mk(10000, 9999, 9999, 0)) == jp.JP_MODE_SEQ_RECOMMENDED   # Gauss-Seidel
+    assert jp.jp_select_mode(L, mk(1000, 999, 999, 0)) == jp.JP_MODE_TLS   # 0.999: not above tau_high
     assert jp.jp_select_mode(L, mk(1000, 0, 0, 0)) == jp.JP_MODE_DOALL
     assert jp.jp_select_mode(cpu_loop(r=False, w=False), None) == jp.JP_MODE_DOALL
 
@@ -263,10 +264,10 @@ def test_plan_matches_oracle_composition(seed):
             tasks.append([s, e, md])
     A = torch.zeros(n, dtype=torch.int32)
     L = jp.Loop(0, 0, n, A, r=torch.zeros(n, dtype=torch.int32), w=torch.zeros(n, dtype=torch.int32))
-    got = jp.jp_plan(L, profs, world, scheme=jp.JP_SCHED_STEALING, chunk_iters=chunk)
+    got = jp.jp_plan(L, profs, world, scheme=jp.JP_SCHED_STEALING, chunk_iters=chunk, tau_high=0.25)
     exp, _ = OS.stealing_plan([tuple(t) for t in tasks], world, chunk, None, 1.0)
     assert [tuple(int(x) for x in r) for r in got] == [tuple(int(x) for x in r) for r in exp]
-    got = jp.jp_plan(L, profs, world, scheme=jp.JP_SCHED_SHARING, chunk_iters=chunk)
+    got = jp.jp_plan(L, profs, world, scheme=jp.JP_SCHED_SHARING, chunk_iters=chunk, tau_high=0.25)
     rg = OS.sharing_ranges(n, [1.0] * world)
     exp = [(max(s, b), min(e, ee), md, k) for k, (b, ee) in enumerate(rg) for s, e, md in tasks
            if max(s, b) < min(e, ee)]
