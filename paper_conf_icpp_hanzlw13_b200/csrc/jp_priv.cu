@@ -151,10 +151,8 @@ __global__ void __launch_bounds__(kPrivThreads) k_priv_tmp_vec(DLoop L, unsigned
 // too, so the check-before-atomic filter keeps working).
 constexpr int kPrivTile = 4096, kPrivStages = 4, kPrivTmaThreads = 256;
 
-// fuse_apply (cooperative launch, one CTA per SM): after every CTA's flush a
-// grid-wide barrier, then the merged keys are applied to T in the same kernel
-// (R1 + R2 in one launch, single-GPU jp_run_privatized only: across GPUs the
-// keys are merged by C4 between the stream and the finalize).
+// (k_priv_tmp_tma is the one-pass stream whose keys are merged by a later C4 and
+// finalize; R1 + R2 in one launch is k_priv_tmp_2ph below.)
 // C4 fused into the stream (jp_priv_stream_merge): every rank's inbox holds
 //   [0] epoch of the last merge, [32 + 2*8] flags[parity][sender] = epoch,
 //   [64 ...] keys[parity][sender][lenT]
@@ -181,13 +179,16 @@ __device__ __forceinline__ unsigned long long gtimer_ns() {
 // Double-buffered by epoch parity: a rank writes parity e+1 only after its
 // merge e, which needed every peer's flag e, i.e. every peer's push e -- pushes
 // of e+1 never land in a buffer a peer still reduces for e-1.
-__device__ void merge_p2p_epilogue(const DLoop &L, const unsigned long long *kT, const MergeP2P &M) {
+struct MergeState { unsigned long long e; int par; };
+
+// push this rank's keys into slot (parity, me) of every rank's inbox and raise
+// one system-scope release flag per peer (CTA 0, all keys in kT)
+__device__ MergeState merge_p2p_push(const DLoop &L, const unsigned long long *kT, const MergeP2P &M) {
   __shared__ unsigned long long e_s;
-  __shared__ int ok;
   unsigned long long *in = M.inbox[M.me];
   const int tid = threadIdx.x, nt = blockDim.x;
   const int64_t lenT = L.lenT;
-  if (tid == 0) { e_s = in[0] + 1; ok = 1; }
+  if (tid == 0) e_s = in[0] + 1;
   __syncthreads();
   const unsigned long long e = e_s;
   const int par = (int)(e & 1);
@@ -201,13 +202,26 @@ __device__ void merge_p2p_epilogue(const DLoop &L, const unsigned long long *kT,
   if (tid < M.world) {
     unsigned long long *f = M.inbox[tid] + kInboxFlags + par * kMergePeers + M.me;
     asm volatile("st.release.sys.global.u64 [%0], %1;" ::"l"(f), "l"(e) : "memory");
-    // ... and wait for sender tid's flag of this epoch here
-    const unsigned long long *g = in + kInboxFlags + par * kMergePeers + tid;
+  }
+  return MergeState{e, par};
+}
+
+// wait for every sender's flag of this epoch, reduce the world tables (local
+// loads) and apply the merged last writers to T (CTA 0)
+__device__ void merge_p2p_finish(const DLoop &L, const MergeP2P &M, MergeState st) {
+  __shared__ int ok;
+  unsigned long long *in = M.inbox[M.me];
+  const int tid = threadIdx.x, nt = blockDim.x;
+  const int64_t lenT = L.lenT;
+  if (tid == 0) ok = 1;
+  __syncthreads();
+  if (tid < M.world) {
+    const unsigned long long *g = in + kInboxFlags + st.par * kMergePeers + tid;
     const unsigned long long t0 = gtimer_ns();
     for (;;) {
       unsigned long long v;
       asm volatile("ld.acquire.sys.global.u64 %0, [%1];" : "=l"(v) : "l"(g) : "memory");
-      if (v >= e) break;
+      if (v >= st.e) break;
       if (gtimer_ns() - t0 > 4000000000ull) { ok = 0; atomicExch(M.err, 1); break; }
       __nanosleep(100);
     }
@@ -215,7 +229,7 @@ __device__ void merge_p2p_epilogue(const DLoop &L, const unsigned long long *kT,
   __syncthreads();
   if (!ok) return;
   asm volatile("fence.acq_rel.sys;" ::: "memory");
-  const unsigned long long *keys = in + kInboxKeys + (int64_t)par * M.world * lenT;
+  const unsigned long long *keys = in + kInboxKeys + (int64_t)st.par * M.world * lenT;
   for (int64_t b = tid; b < lenT; b += nt) {
     unsigned long long m = 0;
     for (int r = 0; r < M.world; r++) {
@@ -225,12 +239,161 @@ __device__ void merge_p2p_epilogue(const DLoop &L, const unsigned long long *kT,
     if (m) L.T[b] = (uint32_t)m;
   }
   __syncthreads();
-  if (tid == 0) in[0] = e;
+  if (tid == 0) in[0] = st.e;
 }
 
-template <int DT, bool MERGE = false>
+// One CTA, after the grid barrier that follows every CTA's key flush: push this
+// rank's keys into slot (parity, me) of every rank's inbox with plain peer
+// stores (posted over NVLink), then one release flag per peer; wait for every
+// sender's flag of this epoch in the local inbox; reduce the world key tables
+// (local loads) and apply the merged last writers to T.  Double-buffered by
+// epoch parity: a rank writes parity e+1 only after its merge e, which needed
+// every peer's flag e, i.e. every peer's push e -- pushes of e+1 never land in
+// a buffer a peer still reduces for e-1.
+__device__ void merge_p2p_epilogue(const DLoop &L, const unsigned long long *kT, const MergeP2P &M) {
+  merge_p2p_finish(L, M, merge_p2p_push(L, kT, M));
+}
+
+// Two phases in one cooperative kernel (config-4 shape, the whole call's run):
+// phase 1 streams s alone -- the index check of reading A13 (out-of-range slots
+// counted into *vbad, nullable) and the per-CTA last-writer table, flushed as
+// packed keys (the value c0*X[i] recomputed at the CTA's last writer of a slot);
+// a grid barrier; then, only if no index was bad, phase 2 streams X into Y =
+// c0*X + c1 and the merged keys reach T -- applied by every CTA (one rank), or,
+// with MERGE, pushed to every rank's inbox by CTA 0 right after the barrier and
+// merged at its end, so the exchange overlaps the Y stream.  s, X and Y each
+// cross HBM once: 12 B/iter, the check included.
+// 4 stages of 32 KiB per phase (the same 128 KiB of shared memory as the one-pass
+// kernel): 16 KiB tiles left each CTA bound by its per-tile barrier / bulk-store
+// turnaround in the X -> Y phase (188 us for config 4, ncu)
+constexpr int kPh = kPrivStages, kPh2Tile = 2 * kPrivTile, kPh2Threads = 1024;
+template <int DT, bool MERGE>
+__global__ void __launch_bounds__(kPh2Threads, 1) k_priv_tmp_2ph(DLoop L, unsigned long long *kT, int64_t ntiles,
+                                                                     int64_t *vbad, MergeP2P M) {
+  extern __shared__ __align__(128) uint32_t psm[];   // [kPh][tile] then tT[lenT]
+  __shared__ __align__(8) unsigned long long full1[kPh], full2[kPh];
+  uint32_t *tT = psm + (size_t)kPh * kPh2Tile;
+  const int tid = threadIdx.x;
+  const uint32_t lenT = (uint32_t)L.lenT;
+  for (int64_t k = tid; k < L.lenT; k += kPh2Threads) tT[k] = 0;
+  const int64_t my = ntiles > blockIdx.x ? (ntiles - 1 - blockIdx.x) / gridDim.x + 1 : 0;
+  auto tile_of = [&](int64_t k) { return ntiles - 1 - (int64_t)blockIdx.x - k * gridDim.x; };
+  auto buf = [&](int64_t k) { return psm + (size_t)(k % kPh) * kPh2Tile; };
+  if (tid == 0) {
+    for (int sg = 0; sg < kPh; sg++) { mbar_init(&full1[sg], 1); mbar_init(&full2[sg], 1); }
+    asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+  }
+  __syncthreads();
+  // ---------------- phase 1: s ----------------
+  auto issue1 = [&](int64_t k) {
+    mbar_expect_tx(&full1[k % kPh], kPh2Tile * 4);
+    bulk_load(buf(k), L.s + tile_of(k) * kPh2Tile, kPh2Tile * 4, &full1[k % kPh]);
+  };
+  if (tid == 0)
+    for (int64_t k = 0; k < kPh && k < my; k++) issue1(k);
+  unsigned bad = 0;
+  for (int64_t k = 0; k < my; k++) {
+    mbar_wait(&full1[k % kPh], (uint32_t)((k / kPh) & 1));
+    const int64_t e0 = tile_of(k) * kPh2Tile;
+    const int4 *S4 = reinterpret_cast<const int4 *>(buf(k));
+    // the slot table's current values are read for all of a thread's iterations
+    // first, then the (rare, with the descending walk) atomics issued: a stale
+    // read only costs an extra atomicMax, and the loads no longer wait behind
+    // possibly aliasing atomics one by one
+    constexpr int kQ = kPh2Tile / 4 / kPh2Threads;
+    int sl[4 * kQ];
+    uint32_t cur[4 * kQ];
+#pragma unroll
+    for (int q = 0; q < kQ; q++) {
+      const int4 sv = S4[kPh2Tile / 4 - 1 - (q * kPh2Threads + tid)];   // descending in the tile
+      sl[4 * q + 0] = sv.w; sl[4 * q + 1] = sv.z; sl[4 * q + 2] = sv.y; sl[4 * q + 3] = sv.x;
+    }
+#pragma unroll
+    for (int m = 0; m < 4 * kQ; m++) {
+      const bool ok = (uint32_t)sl[m] < lenT;
+      bad += !ok;
+      cur[m] = ok ? tT[sl[m]] : 0xFFFFFFFFu;
+    }
+#pragma unroll
+    for (int m = 0; m < 4 * kQ; m++) {
+      const int q = m >> 2;
+      const int64_t i = e0 + 4 * (kPh2Tile / 4 - 1 - (q * kPh2Threads + tid)) + (3 - (m & 3));
+      const uint32_t v = (uint32_t)(i + 1);
+      if (cur[m] < v) atomicMax(&tT[sl[m]], v);
+    }
+    __syncthreads();   // the stage is read: refill it
+    if (tid == 0 && k + kPh < my) issue1(k + kPh);
+  }
+  if (blockIdx.x == 0)   // element tail [ntiles * tile, n)
+    for (int64_t i = ntiles * kPh2Tile + tid; i < L.n; i += kPh2Threads) {
+      const int32_t sv = L.s[i];
+      if ((uint32_t)sv < lenT) smem_last(tT, sv, i); else bad++;
+    }
+  bad = __reduce_add_sync(0xffffffffu, bad);
+  if (vbad && (tid & 31) == 0 && bad) atomicAdd(reinterpret_cast<unsigned long long *>(vbad), (unsigned long long)bad);
+  __syncthreads();
+  for (int64_t b = tid; b < L.lenT; b += kPh2Threads) {
+    const uint32_t e = tT[b];
+    if (e) atomicMax(&kT[b], pack_key(L.base + e - 1, op_mul<DT>(L.c0, __ldg(L.X + e - 1))));
+  }
+  cg::this_grid().sync();   // every CTA's keys are in, every index checked
+  if (vbad && *reinterpret_cast<volatile int64_t *>(vbad)) return;   // nothing written (reading A13)
+  MergeState ms{};
+  if constexpr (MERGE) {
+    if (blockIdx.x == 0) ms = merge_p2p_push(L, kT, M);
+  } else {
+    for (int64_t b = (int64_t)blockIdx.x * kPh2Threads + tid; b < L.lenT; b += (int64_t)gridDim.x * kPh2Threads) {
+      const unsigned long long key = __ldcg(&kT[b]);
+      if (key) L.T[b] = (uint32_t)key;
+    }
+  }
+  // ---------------- phase 2: X -> Y ----------------
+  auto issue2 = [&](int64_t k) {
+    mbar_expect_tx(&full2[k % kPh], kPh2Tile * 4);
+    bulk_load(buf(k), L.X + tile_of(k) * kPh2Tile, kPh2Tile * 4, &full2[k % kPh]);
+  };
+  if (tid == 0)
+    for (int64_t k = 0; k < kPh - 1 && k < my; k++) issue2(k);
+  for (int64_t k = 0; k < my; k++) {
+    mbar_wait(&full2[k % kPh], (uint32_t)((k / kPh) & 1));
+    uint4 *X4 = reinterpret_cast<uint4 *>(buf(k));
+#pragma unroll
+    for (int q = 0; q < kPh2Tile / 4 / kPh2Threads; q++) {
+      const int v = q * kPh2Threads + tid;
+      const uint4 x = X4[v];
+      uint4 y;
+      y.x = op_add<DT>(op_mul<DT>(L.c0, x.x), L.c1);
+      y.y = op_add<DT>(op_mul<DT>(L.c0, x.y), L.c1);
+      y.z = op_add<DT>(op_mul<DT>(L.c0, x.z), L.c1);
+      y.w = op_add<DT>(op_mul<DT>(L.c0, x.w), L.c1);
+      X4[v] = y;
+    }
+    asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
+    __syncthreads();
+    if (tid == 0) {
+      bulk_store(L.A + tile_of(k) * kPh2Tile, buf(k), kPh2Tile * 4);
+      asm volatile("cp.async.bulk.commit_group;" ::: "memory");
+      if (k + kPh - 1 < my) {
+        asm volatile("cp.async.bulk.wait_group.read 1;" ::: "memory");
+        issue2(k + kPh - 1);
+      }
+    }
+  }
+  if (tid == 0) asm volatile("cp.async.bulk.wait_group 0;" ::: "memory");
+  if (blockIdx.x == 0)
+    for (int64_t i = ntiles * kPh2Tile + tid; i < L.n; i += kPh2Threads)
+      L.A[i] = op_add<DT>(op_mul<DT>(L.c0, L.X[i]), L.c1);
+  if constexpr (MERGE) {
+    if (blockIdx.x == 0) merge_p2p_finish(L, M, ms);
+  }
+}
+
+// fuse_apply (cooperative launch): after every CTA's flush a grid barrier, then
+// the keys are applied to T by every CTA (R1 + R2 in one launch when the index
+// check is not needed; k_priv_tmp_2ph carries the check)
+template <int DT>
 __global__ void __launch_bounds__(kPrivTmaThreads, 1) k_priv_tmp_tma(DLoop L, unsigned long long *kT, int64_t ntiles,
-                                                                     int fuse_apply, MergeP2P M = MergeP2P{}) {
+                                                                     int fuse_apply) {
   if (aborted(L)) return;
   extern __shared__ __align__(128) uint32_t psm[];   // [stage][2][tile] then tT[lenT]
   __shared__ __align__(8) unsigned long long full[kPrivStages];
@@ -304,10 +467,6 @@ __global__ void __launch_bounds__(kPrivTmaThreads, 1) k_priv_tmp_tma(DLoop L, un
   }
   if (fuse_apply) {
     cg::this_grid().sync();   // every CTA's keys are in
-    if constexpr (MERGE) {   // C4 across the ranks, then R2, in CTA 0
-      if (blockIdx.x == 0) merge_p2p_epilogue(L, kT, M);
-      return;
-    }
     for (int64_t b = (int64_t)blockIdx.x * kPrivTmaThreads + tid; b < L.lenT; b += (int64_t)gridDim.x * kPrivTmaThreads) {
       const unsigned long long k = __ldcg(&kT[b]);
       if (k) L.T[b] = (uint32_t)k;
@@ -352,22 +511,37 @@ static void run_priv(const DLoop &d0, unsigned long long *kA, unsigned long long
       if (doall_kernel_choice() == 1) {   // bulk-copy staged (the DOALL kernel choice covers both streams)
         const int64_t ntiles = d.n / kPrivTile;
         const size_t smem = (size_t)kPrivStages * 2 * kPrivTile * 4 + (size_t)d.lenT * 4;
-        cudaFuncSetAttribute(k_priv_tmp_tma<DT, false>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+        cudaFuncSetAttribute(k_priv_tmp_tma<DT>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
         int g = num_sms();
         if (max_ctas > 0 && g > max_ctas) g = max_ctas;
         if (ntiles < g) g = (int)(ntiles < 1 ? 1 : ntiles);
-        int fuse = fuse_apply ? 1 : 0;
-        if (fuse) {   // one CTA per SM: co-resident, as a cooperative launch requires
+        if (fuse_apply && !vbad) {   // R1 + R2 in one pass (cooperative: one CTA per SM, co-resident)
           DLoop dd = d;
           int64_t nt = ntiles;
-          validate_first();
+          int fuse = 1;
+          void *args[] = {&dd, &kT, &nt, &fuse};
+          cudaLaunchCooperativeKernel((void *)k_priv_tmp_tma<DT>, dim3(g), dim3(kPrivTmaThreads), args, smem, st);
+          *applied = true;
+        } else if (fuse_apply) {   // with the index check: two phases (s, then X -> Y)
+          const int64_t ntiles = d.n / kPh2Tile;
+          int g = num_sms();
+          if (max_ctas > 0 && g > max_ctas) g = max_ctas;
+          if (ntiles < g) g = (int)(ntiles < 1 ? 1 : ntiles);
+          // two phases: s (index check + last writers), grid barrier, X -> Y and T;
+          // the check of reading A13 needs no pass of its own (s crosses HBM once)
+          DLoop dd = d;
+          dd.abort = nullptr;
+          int64_t nt = ntiles;
+          int64_t *vb = vbad;
+          if (vb) cudaMemsetAsync(vb, 0, sizeof(int64_t), st);
           MergeP2P none{};
-          void *args[] = {&dd, &kT, &nt, &fuse, &none};
-          cudaLaunchCooperativeKernel((void *)k_priv_tmp_tma<DT, false>, dim3(g), dim3(kPrivTmaThreads), args, smem, st);
+          void *args[] = {&dd, &kT, &nt, &vb, &none};
+          cudaFuncSetAttribute(k_priv_tmp_2ph<DT, false>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+          cudaLaunchCooperativeKernel((void *)k_priv_tmp_2ph<DT, false>, dim3(g), dim3(kPh2Threads), args, smem, st);
           *applied = true;
         } else {
           validate_first();
-          k_priv_tmp_tma<DT, false><<<g, kPrivTmaThreads, smem, st>>>(d, kT, ntiles, 0, MergeP2P{});
+          k_priv_tmp_tma<DT><<<g, kPrivTmaThreads, smem, st>>>(d, kT, ntiles, 0);
         }
         note_launch();
         return;
@@ -408,8 +582,8 @@ cudaError_t launch_priv_stream_merge(const Job &j, unsigned long long *kT, unsig
   d.A += d.ioff; d.lenA -= d.ioff;
   d.ioff = 0;
   cudaMemsetAsync(kT, 0, 8 * (size_t)d.lenT, st);
-  const int64_t ntiles = d.n / kPrivTile;
-  const size_t smem = (size_t)kPrivStages * 2 * kPrivTile * 4 + (size_t)d.lenT * 4;
+  const int64_t ntiles = d.n / kPh2Tile;
+  const size_t smem = (size_t)kPh * kPh2Tile * 4 + (size_t)d.lenT * 4;
   cudaError_t e;
   auto go = [&](auto kern) {
     cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
@@ -420,13 +594,13 @@ cudaError_t launch_priv_stream_merge(const Job &j, unsigned long long *kT, unsig
     M.world = world;
     M.me = me;
     M.err = err;
-    int fuse = 1;
     int64_t nt = ntiles;
-    void *args[] = {&d, &kT, &nt, &fuse, &M};
-    e = cudaLaunchCooperativeKernel((const void *)kern, dim3(g), dim3(kPrivTmaThreads), args, smem, st);
+    int64_t *vb = nullptr;   // (the ranks' indices were checked by the partitioned profile)
+    void *args[] = {&d, &kT, &nt, &vb, &M};
+    e = cudaLaunchCooperativeKernel((const void *)kern, dim3(g), dim3(kPh2Threads), args, smem, st);
   };
-  if (j.dt == JP_F32) go(k_priv_tmp_tma<JP_F32, true>);
-  else go(k_priv_tmp_tma<JP_I32, true>);
+  if (j.dt == JP_F32) go(k_priv_tmp_2ph<JP_F32, true>);
+  else go(k_priv_tmp_2ph<JP_I32, true>);
   note_launch();
   if (e != cudaSuccess) return e;
   return launch_check();
