@@ -870,6 +870,24 @@ def run_jp(args):
     e2e["frac_of_copy_bound"] = e2e["value"] / (N2 / tc)
     del stage, hA, hX
     launches_all = int(sum_over_ranks(launches, world, dev))
+    # C7: gathering the sharded output on rank 0 is reported
+    # separately and is not in T(k)
+    gather = None
+    if world > 1:
+        try:
+            outs = [torch.empty_like(wl.A) for _ in range(world)] if rank == 0 else None
+            barrier(world)
+            g0, g1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            g0.record(st)
+            torch.distributed.gather(wl.A, outs, dst=0)
+            g1.record(st)
+            barrier(world)
+            gms = max_over_ranks(g0.elapsed_time(g1), world, dev)
+            gather = {"ms": gms, "bytes_to_rank0": 4 * (N2 - (s1 - s0)), "GBps": 4 * (N2 - (s1 - s0)) / (gms * 1e-3) / 1e9,
+                      "what": "torch.distributed.gather of every rank's Y shard to rank 0 (C7), after the timed steps"}
+            del outs
+        except Exception as ex:   # e.g. the gloo test mode with device tensors
+            gather = {"error": repr(ex)[:200]}
 
     out = None
     if rank == 0:
@@ -886,7 +904,8 @@ def run_jp(args):
                                               "(profiles/ncu_doall_traffic.json, N=1), x this rank's share",
                             "algorithmic_bytes_per_iter": BYTES_PER_ITER_SAXPY, "peak_source": peak_src,
                             "kernel_ms": kernel_ms},
-               "clocks": clk.summary(), "e2e": e2e, "gpu_launches": launches_all, "paper_context": PAPER_CONTEXT}
+               "clocks": clk.summary(), "e2e": e2e, "gpu_launches": launches_all, "paper_context": PAPER_CONTEXT,
+               "gather_to_one": gather}
     if not args.no_modes:
         del wl, L
         torch.cuda.empty_cache()

@@ -36,7 +36,19 @@ namespace cg = cooperative_groups;
 
 namespace jp {
 
-constexpr int kFlowT = 512, kFlowK = 8;
+// CTA shape (measured on config 3, whole jp_schedule, d = 0.1/1/5/10%: 512 x 8 x 1
+// CTA/SM 0.738/0.746/0.812/0.880 ms; 512 x 4 x 2 0.743/0.736/0.788/0.856; 1024 x 4
+// 0.746/0.742/0.797/0.857; 256 x 8 x 3 0.770/0.778/0.865/0.947): random-access bound
+#ifndef JP_FLOW_T
+#define JP_FLOW_T 512
+#endif
+#ifndef JP_FLOW_K
+#define JP_FLOW_K 4
+#endif
+#ifndef JP_FLOW_MINB
+#define JP_FLOW_MINB 2
+#endif
+constexpr int kFlowT = JP_FLOW_T, kFlowK = JP_FLOW_K;
 constexpr unsigned long long kFlowTag = 1ull << 32;
 constexpr long long kFlowSpinLimit = 1ll << 22;   // a lost writer (inconsistent guide) ends the wait with an error
 
@@ -116,7 +128,7 @@ struct Flow {
 };
 
 template <int DT>
-__global__ void __launch_bounds__(kFlowT, 1) k_tls_flow(DLoop L, const uint32_t *graw, const uint32_t *gsrc,
+__global__ void __launch_bounds__(kFlowT, JP_FLOW_MINB) k_tls_flow(DLoop L, const uint32_t *graw, const uint32_t *gsrc,
                                                        unsigned long long *V, int64_t *stats) {
   Flow<DT> F;
   F.L = L; F.graw = graw; F.gsrc = gsrc; F.V = V;
@@ -152,7 +164,7 @@ static cudaError_t run_flow(const Job &j, const uint32_t *graw, const uint32_t *
   int maxb = 0;
   cudaOccupancyMaxActiveBlocksPerMultiprocessor(&maxb, (const void *)k_tls_flow<DT>, kFlowT, 0);
   if (maxb < 1) return cudaErrorInvalidConfiguration;
-  int grid = num_sms();
+  int grid = num_sms() * maxb;
   const int64_t need = (j.d.n + kFlowT - 1) / kFlowT;
   if (need < grid) grid = (int)(need < 1 ? 1 : need);
   DLoop d = j.d;
