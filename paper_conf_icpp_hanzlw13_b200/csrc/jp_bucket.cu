@@ -10,7 +10,7 @@
 // accesses are first PARTITIONED by address instead, so every first-writer /
 // first-reader table lives in one CTA's shared memory:
 //
-//   count    per tile of 4096 iterations: accesses per bucket of 8192
+//   count    per tile of 16384 iterations: accesses per bucket of 8192
 //            addresses (shared-memory histogram), and the out-of-range count;
 //   scan     per bucket, the tiles' exclusive offsets; then the buckets' bases;
 //   scatter  every access as an 8-byte record (iteration, address in its
@@ -40,9 +40,9 @@ namespace jp {
 
 constexpr int kBShift = 13;                 // addresses per bucket: 8192
 constexpr int kBSpan = 1 << kBShift;
-constexpr int kTShift = 12;                 // iterations per tile: 4096
+constexpr int kTShift = 14;                 // iterations per tile: 16384
 constexpr int kTile = 1 << kTShift;
-constexpr int kBThreads = 512;
+constexpr int kBThreads = 1024;
 constexpr int kEvalThreads = 512;
 constexpr int kMaxBuckets = 8192;           // len_A <= 2^26
 constexpr int kMaxTiles = 16384;            // n <= 2^26
@@ -193,9 +193,12 @@ __global__ void __launch_bounds__(1024) k_bk_scan_buckets(const uint32_t *tot, i
 template <int OP>
 __global__ void __launch_bounds__(kBThreads) k_bk_scatter(BkView V, int vec, const uint32_t *off, const uint32_t *tot,
                                                          const uint32_t *base, unsigned long long *rec) {
-  extern __shared__ unsigned long long sm64[];
-  unsigned long long *stage = sm64;                            // [2 * kTile] il | a << 12 | write << 63
-  uint32_t *lpos = reinterpret_cast<uint32_t *>(stage + 2 * kTile);   // [B + 1] local exclusive starts
+  // staging: 6 bytes per record -- il | address in the bucket << 14 | write << 31,
+  // and the bucket (16 bits) -- so that a 16384-iteration tile fits one SM
+  extern __shared__ uint32_t sm32[];
+  uint32_t *stage = sm32;                                      // [2 * kTile]
+  uint16_t *stb = reinterpret_cast<uint16_t *>(stage + 2 * kTile);      // [2 * kTile]
+  uint32_t *lpos = reinterpret_cast<uint32_t *>(stb + 2 * kTile);       // [B + 1] local exclusive starts
   uint32_t *cur = lpos + V.B + 1;                              // [B]
   uint32_t *gpos = cur + V.B;                                  // [B] global start of this tile's run
   __shared__ uint32_t wsum[kBThreads / 32];
@@ -251,8 +254,10 @@ __global__ void __launch_bounds__(kBThreads) k_bk_scatter(BkView V, int vec, con
     for (int m = 0; m < kA; m++) {
       const int k = OP == JP_OP_ADD_C ? m >> 1 : m;
       const bool wr = OP == JP_OP_ADD_C ? (m & 1) == 0 : true;
-      if (k < kn)
-        stage[pos[m]] = (unsigned long long)(il0 + k) | (unsigned long long)a[m] << kTShift | (wr ? kRecW : 0ull);
+      if (k < kn) {
+        stage[pos[m]] = (uint32_t)(il0 + k) | (a[m] & (kBSpan - 1)) << kTShift | (wr ? 1u << 31 : 0u);
+        stb[pos[m]] = (uint16_t)(a[m] >> kBShift);
+      }
     }
   });
   __syncthreads();
@@ -262,10 +267,9 @@ __global__ void __launch_bounds__(kBThreads) k_bk_scatter(BkView V, int vec, con
   __syncthreads();
   const uint32_t nrec = lpos[B];
   for (uint32_t k = threadIdx.x; k < nrec; k += kBThreads) {
-    const unsigned long long x = stage[k];
-    const uint32_t a = (uint32_t)(x >> kTShift) & 0x7FFFFFFFu;
-    rec[k + gpos[a >> kBShift]] = (unsigned long long)(i0 + ((uint32_t)x & (kTile - 1))) |
-                                  (unsigned long long)(a & (kBSpan - 1)) << 32 | (x & kRecW);
+    const uint32_t x = stage[k];
+    rec[k + gpos[stb[k]]] = (unsigned long long)(i0 + (x & (kTile - 1))) |
+                            (unsigned long long)((x >> kTShift) & (kBSpan - 1)) << 32 | (x >> 31 ? kRecW : 0ull);
   }
 }
 
@@ -434,7 +438,7 @@ void run_bucket(const BkPlan &P, const DLoop &d, int64_t *hdr, BkOut O, cudaStre
   k_bk_count<OP><<<T, kBThreads, 4 * (size_t)B, st>>>(P.v, vec, P.cnt, &hdr[H_BAD]);
   k_bk_scan_tiles<<<(B + 31) / 32, 1024, 0, st>>>(P.cnt, T, B, P.tot);
   k_bk_scan_buckets<<<1, 1024, 0, st>>>(P.tot, B, P.base);
-  const size_t ssm = 8 * 2 * (size_t)kTile + 4 * (3 * (size_t)B + 1);
+  const size_t ssm = 6 * 2 * (size_t)kTile + 4 * (3 * (size_t)B + 1);
   cudaFuncSetAttribute(k_bk_scatter<OP>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)ssm);
   k_bk_scatter<OP><<<T, kBThreads, ssm, st>>>(P.v, vec, P.cnt, P.tot, P.base, P.rec);
   const int nch = O.cc ? (int)((d.n + O.chunk - 1) / O.chunk) : 0;
