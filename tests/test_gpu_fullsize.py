@@ -130,3 +130,43 @@ def test_doall_indirect_multi_trip(op, dt, generic, monkeypatch):
     assert equal_bytes(g.A, A), first_diff(g.A, A)
     if T is not None:
         assert equal_bytes(g.T, T)
+
+
+@pytest.mark.parametrize("d,delta", [(0.01, 1024), (0.10, 1024), (0.01, 1 << 20), (0.10, 1 << 20)])
+def test_config3_waw_full_size_restart(d, delta):
+    """Config 3's shape with write-after-write (on-chip recovery illegal), N = 2^24,
+    through jp_schedule -- the bench's config3_waw rows: restart TLS under the
+    distance-steered cap; every byte of A and the statistics of jpo_sim_tls under
+    that cap."""
+    wl = synth.config3_waw(d, delta=delta)
+    ref = to_oracle(wl)
+    g = wl.to(DEV)
+    L = jp.Loop.from_workload(g)
+    res = jp.jp_schedule(L, jp.workspace(L))
+    torch.cuda.synchronize()
+    assert res["mode"] == jp.JP_MODE_TLS and res["tls_recovery"] == jp.JP_TLS_RESTART, res
+    p = O.profile(ref)
+    assert (res["prof"]["raw_iters"], res["prof"]["waw_iters"]) == (p["raw_iters"], p["waw_iters"])
+    st, A, _, stats = O.sim_tls(ref, 0, res["tls_w_max"], p["raw_iters"])
+    assert equal_bytes(g.A, A), first_diff(g.A, A)
+    assert res["tls"] == stats, (res["tls"], stats)
+
+
+@pytest.mark.parametrize("split", [3, 5])
+def test_schedule_ranges_of_config3(split):
+    """A loop run as consecutive ranges (iter_base = ident_off = the range start),
+    each through jp_schedule on the shared arrays -- the address-bucket profile,
+    Fig. 2(b) and the one-window on-chip TLS of every range use global ids; the
+    final A is the sequential one (ranges in order = program order)."""
+    n = (1 << 21) + 13
+    wl = synth.config3(0.05, n=n)
+    _, A, _ = O.run_seq(to_oracle(wl))
+    g = wl.to(DEV)
+    full = jp.Loop.from_workload(g)
+    cuts = [n * k // split for k in range(split + 1)]
+    for b, e in zip(cuts[:-1], cuts[1:]):
+        part = full.range(b, e)
+        res = jp.jp_schedule(part, jp.workspace(part))
+        torch.cuda.synchronize()
+        assert res["mode"] in (jp.JP_MODE_TLS, jp.JP_MODE_DOALL, jp.JP_MODE_PRIVATIZED), res
+    assert equal_bytes(g.A, A), first_diff(g.A, A)
