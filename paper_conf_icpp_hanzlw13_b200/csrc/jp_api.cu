@@ -110,6 +110,7 @@ SchedLayout sched_layout(const jp_loop *L) {
   s.conf = o; o = al256(o + 8 * kMaxTasks);
   s.tstats = o; o = al256(o + 32 * kMaxTasks);
   s.ranges = o; o = al256(o + 16 * kMaxTasks);
+  s.crange = o; o = al256(o + 8 * (size_t)nck);
   s.total = o;
   return s;
 }
@@ -1243,9 +1244,12 @@ static std::vector<Task> chunk_tasks(const int64_t *hc, int64_t n, int64_t chunk
 // conf[u] bit t: tasks t and u touch a common address, at least one writing it (reading B2); syncs
 // ranges_out (nullable): the per-task address ranges of the prefilter
 // ([4][kMaxTasks]: minA, maxA, minT, maxT) when it ran, else left empty
+// chunk_rg (nullable): per chunk the min / max address of A it touches (the bucket
+// profile's), from which the task ranges follow without the k_task_ranges pass
 static jp_status task_conflicts(const Job &j, const jp_loop *L, void *ws, const Layout &lo,
                                 const std::vector<Task> &tasks, int64_t chunk, std::vector<unsigned long long> &conf,
-                                cudaStream_t st, std::vector<uint32_t> *ranges_out = nullptr) {
+                                cudaStream_t st, std::vector<uint32_t> *ranges_out = nullptr,
+                                const std::vector<uint32_t> *chunk_rg = nullptr) {
   const int nt = (int)tasks.size();
   if (ranges_out) ranges_out->clear();
   conf.assign(kMaxTasks, 0);
@@ -1260,11 +1264,20 @@ static jp_status task_conflicts(const Job &j, const jp_loop *L, void *ws, const 
   JP_CUDA(cudaMemcpyAsync(dct, ct.data(), 4 * nck, cudaMemcpyHostToDevice, st), "task map H2D");
   // cheap sufficient test first: tasks with disjoint address ranges in every array never conflict
   if (!getenv("JP_TASK_MASKS_ALWAYS")) {
-    uint32_t *drg = reinterpret_cast<uint32_t *>(sch + sl.ranges);
-    JP_CUDA(launch_task_ranges(j, dct, chunk, drg, st), "task ranges");
     std::vector<uint32_t> rg(4 * kMaxTasks);
-    JP_CUDA(cudaMemcpyAsync(rg.data(), drg, 16 * kMaxTasks, cudaMemcpyDeviceToHost, st), "ranges D2H");
-    JP_CUDA(cudaStreamSynchronize(st), "ranges sync");
+    if (chunk_rg && (j.op == JP_OP_ADD_C || j.op == JP_OP_SAXPY)) {   // A only: the T ranges stay empty
+      for (int t = 0; t < kMaxTasks; t++) { rg[t] = rg[2 * kMaxTasks + t] = 0xFFFFFFFFu; rg[kMaxTasks + t] = rg[3 * kMaxTasks + t] = 0; }
+      for (int t = 0; t < nt; t++)
+        for (int64_t k = tasks[t].s / chunk; k * chunk < tasks[t].e; k++) {
+          rg[t] = std::min(rg[t], (*chunk_rg)[2 * k]);
+          rg[kMaxTasks + t] = std::max(rg[kMaxTasks + t], (*chunk_rg)[2 * k + 1]);
+        }
+    } else {
+      uint32_t *drg = reinterpret_cast<uint32_t *>(sch + sl.ranges);
+      JP_CUDA(launch_task_ranges(j, dct, chunk, drg, st), "task ranges");
+      JP_CUDA(cudaMemcpyAsync(rg.data(), drg, 16 * kMaxTasks, cudaMemcpyDeviceToHost, st), "ranges D2H");
+      JP_CUDA(cudaStreamSynchronize(st), "ranges sync");
+    }
     if (ranges_out) *ranges_out = rg;
     auto ov = [&](int a, int t, int u) {   // array a: 0 A, 1 T
       const uint32_t *mn = rg.data() + 2 * a * kMaxTasks, *mx = mn + kMaxTasks;
@@ -1304,9 +1317,20 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
   // the first all-SM TLS task finds this call's pair table in the write-log
   // region: it needs no reset (see launch_tls_fwd_grid); later ones do
   bool s_fresh = pairs;
+  // the writer of every raw read, recorded by the bucket profile (ADD_C with the
+  // guide): lets a write-once, WAR-free TLS task run as one window (path 8) even
+  // when some of its reads were written by an earlier task.  Kept in region 7
+  // (the write log of paths 5 / 6, unused by path 8)
+  int32_t *wsrc = nullptr;
+  uint32_t *crange = nullptr;   // per-chunk address ranges from the bucket profile (task PDG prefilter)
   if (bucket_profile_ok(j, ws, lo)) {   // large A: the profile by address buckets (jp_bucket.cu)
     s_fresh = false;                    // (region 7 is not filled: the TLS task resets it)
-    JP_CUDA(launch_prof_bucket(j, ws, lo, gbits, gbits ? gbits + (L->n + 31) / 32 : nullptr, chunk, cc, st),
+    if (gbits && j.op == JP_OP_ADD_C && lo.bytes[R_TLS_S_A] >= 4 * (size_t)L->n && !getenv("JP_TLS_NO_FLOW"))
+      wsrc = at<int32_t>(ws, lo, R_TLS_S_A);
+    if (chunk % kBucketTile == 0 && !getenv("JP_TASK_MASKS_ALWAYS"))
+      crange = reinterpret_cast<uint32_t *>(sch + sl.crange);
+    JP_CUDA(launch_prof_bucket(j, ws, lo, gbits, gbits ? gbits + (L->n + 31) / 32 : nullptr, chunk, cc, st, wsrc,
+                               crange),
             "profile (buckets)");
   } else {
     JP_CUDA(launch_prof_stamp(j, ws, lo, st, pairs), "profile stamp");
@@ -1314,7 +1338,12 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
             "profile classify");
   }
   std::vector<int64_t> hc(3 * nck), h(8);
+  std::vector<uint32_t> hcr;
   JP_CUDA(cudaMemcpyAsync(hc.data(), cc, 24 * nck, cudaMemcpyDeviceToHost, st), "chunk D2H");
+  if (crange) {
+    hcr.resize(2 * nck);
+    JP_CUDA(cudaMemcpyAsync(hcr.data(), crange, 8 * nck, cudaMemcpyDeviceToHost, st), "chunk ranges D2H");
+  }
   JP_CUDA(cudaMemcpyAsync(h.data(), at<int64_t>(ws, lo, R_HEADER), 64, cudaMemcpyDeviceToHost, st), "profile D2H");
   JP_CUDA(cudaStreamSynchronize(st), "profile sync");
   if (h[H_BAD]) return fail(JP_ERR_INDEX, "%lld index entries are outside their arrays", (long long)h[H_BAD]);
@@ -1328,7 +1357,7 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
   // 3. inter-task conflicts (PDG) and topological batches
   std::vector<unsigned long long> conf(kMaxTasks, 0);
   std::vector<uint32_t> trg;
-  JP_TRY(task_conflicts(j, L, ws, lo, tasks, chunk, conf, st, &trg));
+  JP_TRY(task_conflicts(j, L, ws, lo, tasks, chunk, conf, st, &trg, crange ? &hcr : nullptr));
   std::vector<int> level(nt, 0);
   int nlev = nt ? 1 : 0;
   for (int u = 0; u < nt; u++) {
@@ -1345,6 +1374,8 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
   // its writers of raw-read addresses are first writers)
   const bool guided_ok = gfuse;
   std::vector<int> grid_tls;   // on-chip TLS tasks, run on every SM after the batch's other tasks
+  std::vector<int> flow_tasks;  // ... of them, run as one window (path 8): stats completed on the host
+  bool v_zeroed = false;
   cudaEvent_t ev0;
   JP_CUDA(cudaEventCreateWithFlags(&ev0, cudaEventDisableTiming), "event");
   std::vector<cudaEvent_t> evs;
@@ -1435,6 +1466,30 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
       if (level[t] != lv) continue;
       // guided by the whole loop's bitmaps (the task starts on a chunk boundary, a multiple of 32)
       Job sj = sub_job(j, tasks[t].s, tasks[t].e);
+      int64_t twar = 0;
+      for (int64_t k = tasks[t].s / chunk; k * chunk < tasks[t].e; k++) twar += hc[3 * k + 1];
+      if (wsrc && guided_ok && twar == 0 && c.tls_window == 0) {
+        // write-once, WAR-free ADD_C task: one window, DC from the guide (path 8);
+        // reads whose writer precedes the task see A (wsrc)
+        const uint32_t *gb = at<uint32_t>(ws, lo, R_GUIDE);
+        const int64_t nw = (L->n + 31) / 32;
+        auto *V = at<unsigned long long>(ws, lo, R_TLS_C_A);
+        if (!v_zeroed) {
+          cudaMemsetAsync(V, 0, lo.bytes[R_TLS_C_A], st);
+          v_zeroed = true;
+        }
+        JP_CUDA(launch_tls_flow(sj, gb + tasks[t].s / 32, gb + nw + tasks[t].s / 32, V, tstats + 4 * t, st,
+                                wsrc + tasks[t].s, tasks[t].s),
+                "tls task (one window)");
+        flow_tasks.push_back(t);
+        res->tls_w_max = sj.d.n;
+        res->tls_path = 8;
+        res->tls_recovery = JP_TLS_ONCHIP;
+        res->tls_cluster = num_sms();
+        res->tls_guided = 1;
+        tls_tasks.push_back(t);
+        continue;
+      }
       TlsPlan tp;
       jp_profile tprof{};
       tprof.n = sj.d.n;
@@ -1475,6 +1530,14 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
     int64_t s4[4];
     JP_CUDA(cudaMemcpyAsync(s4, tstats + 4 * t, sizeof s4, cudaMemcpyDeviceToHost, st), "tls stats D2H");
     JP_CUDA(cudaStreamSynchronize(st), "tls stats sync");
+    if (std::find(flow_tasks.begin(), flow_tasks.end(), t) != flow_tasks.end()) {
+      // path 8 on the device: s4[3] violations, s4[1] warps that lost their writer
+      if (s4[1]) return fail(JP_ERR_ARG, "one-window TLS task: a violator's writer never published");
+      const int64_t tn = tasks[t].e - tasks[t].s;
+      s4[0] = tn;
+      s4[1] = tn + s4[3];
+      s4[2] = tn > 0 ? 1 : 0;
+    }
     res->tls.committed += s4[0]; res->tls.executed += s4[1]; res->tls.windows += s4[2]; res->tls.violations += s4[3];
   }
   JP_CUDA(cudaStreamSynchronize(st), "schedule sync");

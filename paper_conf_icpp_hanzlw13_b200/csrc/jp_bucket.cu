@@ -55,6 +55,8 @@ struct BkView {
   int64_t n, ioff;
   uint32_t lenA;
   int B, T;
+  uint32_t *crange;       // nullable: per chunk min / max address (chunk = ctiles tiles)
+  int ctiles;
 };
 
 __device__ __forceinline__ int4 ld_idx4(const int32_t *p, int64_t i, int64_t n, int64_t ioff, bool vec) {
@@ -108,6 +110,7 @@ __global__ void __launch_bounds__(kBThreads) k_bk_count(BkView V, int vec, uint3
   for (int b = threadIdx.x; b < V.B; b += kBThreads) h[b] = 0;
   __syncthreads();
   unsigned nbad = 0;
+  uint32_t mn = 0xFFFFFFFFu, mx = 0u;   // the tile's address range (crange: a tile lies in one chunk)
   // an out-of-range index is counted (the profile then fails) and filed under
   // bucket 0, consistently with the scatter below
   for_tile<OP>(V, vec, [&](const int4 &w4, const int4 &r4, int, int kn) {
@@ -115,18 +118,31 @@ __global__ void __launch_bounds__(kBThreads) k_bk_count(BkView V, int vec, uint3
     for (int k = 0; k < 4; k++) {
       if (k < kn) {
         const uint32_t a = (uint32_t)q4(w4, k);
-        nbad += a >= V.lenA;
-        atomicAdd(&h[a < V.lenA ? a >> kBShift : 0], 1u);
+        const bool oka = a < V.lenA;
+        nbad += !oka;
+        atomicAdd(&h[oka ? a >> kBShift : 0], 1u);
+        if (oka) { mn = min(mn, a); mx = max(mx, a); }
         if constexpr (OP == JP_OP_ADD_C) {
           const uint32_t c = (uint32_t)q4(r4, k);
-          nbad += c >= V.lenA;
-          atomicAdd(&h[c < V.lenA ? c >> kBShift : 0], 1u);
+          const bool okc = c < V.lenA;
+          nbad += !okc;
+          atomicAdd(&h[okc ? c >> kBShift : 0], 1u);
+          if (okc) { mn = min(mn, c); mx = max(mx, c); }
         }
       }
     }
   });
   nbad = __reduce_add_sync(0xffffffffu, nbad);
   if ((threadIdx.x & 31) == 0 && nbad) atomicAdd(reinterpret_cast<unsigned long long *>(bad), (unsigned long long)nbad);
+  if (V.crange) {
+    mn = __reduce_min_sync(0xffffffffu, mn);
+    mx = __reduce_max_sync(0xffffffffu, mx);
+    if ((threadIdx.x & 31) == 0 && mn <= mx) {
+      const int c = blockIdx.x / V.ctiles;
+      atomicMin(&V.crange[2 * c], mn);
+      atomicMax(&V.crange[2 * c + 1], mx);
+    }
+  }
   __syncthreads();
   uint32_t *row = cnt + (size_t)blockIdx.x * V.B;
   for (int b = threadIdx.x; b < V.B; b += kBThreads) row[b] = h[b];
@@ -279,6 +295,7 @@ struct BkOut {
   int64_t chunk;              // per-chunk counts (cc nullable)
   int64_t *cc;
   int64_t gbase;              // global id of local iteration 0
+  int32_t *wsrc;              // nullable: wsrc[i] = the first writer of raw iteration i's read (ADD_C)
 };
 
 template <int OP>
@@ -343,6 +360,7 @@ __global__ void __launch_bounds__(kEvalThreads) k_bk_eval(BkView V, const uint32
     }
     c_raw += raw; c_war += war; c_waw += waw;
     if (raw) {
+      if (O.wsrc && !(x & kRecW)) O.wsrc[i] = (int32_t)jw;
       if (O.graw) atomicOr(&O.graw[i >> 5], 1u << (i & 31));
       if (O.gsrc) atomicOr(&O.gsrc[jw >> 5], 1u << (jw & 31));
       atomicAdd(&s_dist[31 - __clz(i - jw)], 1u);
@@ -386,6 +404,11 @@ __global__ void __launch_bounds__(kEvalThreads) k_bk_eval(BkView V, const uint32
       if (s_cc[k]) atomicAdd(reinterpret_cast<unsigned long long *>(&O.cc[k]), (unsigned long long)s_cc[k]);
 }
 
+__global__ void k_bk_init_ranges(uint32_t *cr, int64_t nck) {
+  const int64_t c = (int64_t)blockIdx.x * blockDim.x + threadIdx.x;
+  if (c < nck) { cr[2 * c] = 0xFFFFFFFFu; cr[2 * c + 1] = 0u; }
+}
+
 namespace {
 struct BkPlan {
   BkView v;
@@ -422,7 +445,7 @@ bool plan(const Job &j, void *ws, const Layout &lo, BkPlan &P) {
   }
   if (!lo.bytes[R_MINW_A] || rb < 8 * (size_t)nrec) return false;
   if (lo.bytes[R_MAXRX_A] < 4 * ((size_t)T * B + 2 * (size_t)B)) return false;
-  P.v = BkView{d.r, d.w, d.n, d.ioff, (uint32_t)d.lenA, B, T};
+  P.v = BkView{d.r, d.w, d.n, d.ioff, (uint32_t)d.lenA, B, T, nullptr, 1};
   P.rec = at<unsigned long long>(ws, lo, R_MINW_A);
   P.cnt = at<uint32_t>(ws, lo, R_MAXRX_A);
   P.tot = P.cnt + (size_t)T * B;
@@ -455,9 +478,17 @@ bool bucket_profile_ok(const Job &j, void *ws, const Layout &lo) {
 }
 
 cudaError_t launch_prof_bucket(const Job &j, void *ws, const Layout &lo, uint32_t *graw, uint32_t *gsrc,
-                               int64_t chunk, int64_t *cc, cudaStream_t st) {
+                               int64_t chunk, int64_t *cc, cudaStream_t st, int32_t *wsrc, uint32_t *crange) {
   BkPlan P;
   if (!plan(j, ws, lo, P)) return cudaErrorInvalidValue;
+  static_assert(kTile == kBucketTile, "jp_host.h kBucketTile");
+  if (crange && chunk > 0 && chunk % kTile == 0) {
+    const int64_t nck = (j.d.n + chunk - 1) / chunk;
+    k_bk_init_ranges<<<(int)((nck + 255) / 256), 256, 0, st>>>(crange, nck);   // min = ~0, max = 0
+    note_launch();
+    P.v.crange = crange;
+    P.v.ctiles = (int)(chunk / kTile);
+  }
   int64_t *hdr = at<int64_t>(ws, lo, R_HEADER);
   cudaMemsetAsync(hdr, 0, kHeaderBytes, st);
   cudaMemsetAsync(&hdr[H_FIRST_RAW], 0xFF, sizeof(int64_t), st);
@@ -465,7 +496,7 @@ cudaError_t launch_prof_bucket(const Job &j, void *ws, const Layout &lo, uint32_
   if (graw) cudaMemsetAsync(graw, 0, 4 * (size_t)nw, st);
   if (gsrc) cudaMemsetAsync(gsrc, 0, 4 * (size_t)nw, st);
   if (cc) cudaMemsetAsync(cc, 0, sizeof(int64_t) * 3 * ((j.d.n + chunk - 1) / chunk), st);
-  BkOut O{hdr, graw, gsrc, chunk, cc, j.d.base};
+  BkOut O{hdr, graw, gsrc, chunk, cc, j.d.base, j.op == JP_OP_ADD_C ? wsrc : nullptr};
   if (j.op == JP_OP_ADD_C) run_bucket<JP_OP_ADD_C>(P, j.d, hdr, O, st);
   else run_bucket<JP_OP_SAXPY>(P, j.d, hdr, O, st);
   return launch_check();

@@ -33,7 +33,7 @@ constexpr double kTauHigh = 0.999;
 constexpr int kMaxTasks = 64;
 // scheduler scratch sub-layout (inside R_SCHED)
 struct SchedLayout {
-  size_t counts, chunk_task, wmA, rmA, wmT, rmT, conf, tstats, ranges, total;
+  size_t counts, chunk_task, wmA, rmA, wmT, rmT, conf, tstats, ranges, crange, total;
 };
 SchedLayout sched_layout(const jp_loop *L);
 
@@ -67,10 +67,18 @@ bool stamp_pairs_ok(const Job &j, void *ws, const Layout &lo);
 bool bucket_profile_ok(const Job &j, void *ws, const Layout &lo);
 // one-window on-chip TLS (path 8, jp_tls_flow.cu): ADD_C loops with a profile
 // showing waw = war = 0 and the guide words of that profile; stats as noted there
+// wsrc (nullable) with lo: a range [lo, lo + n) of a loop whose profile recorded the
+// writer of every raw read (loop-local ids, wsrc indexed by the range's local i):
+// a raw read whose writer precedes the range reads A (committed) and is no violator
 cudaError_t launch_tls_flow(const Job &j, const uint32_t *graw, const uint32_t *gsrc, unsigned long long *V,
-                            int64_t *stats, cudaStream_t st);
+                            int64_t *stats, cudaStream_t st, const int32_t *wsrc = nullptr, int64_t lo = 0);
+// wsrc (nullable, ADD_C): the first writer of every raw iteration's read (int32 [n])
+// crange (nullable, needs chunk % 16384 == 0): per chunk the min and max address of A
+// the chunk touches (uint32 [2 * chunks]) -- the stealing scheduler's task ranges
 cudaError_t launch_prof_bucket(const Job &j, void *ws, const Layout &lo, uint32_t *graw, uint32_t *gsrc,
-                               int64_t chunk, int64_t *cc, cudaStream_t st);
+                               int64_t chunk, int64_t *cc, cudaStream_t st, int32_t *wsrc = nullptr,
+                               uint32_t *crange = nullptr);
+constexpr int64_t kBucketTile = 16384;   // (jp_bucket.cu's tile: chunk ranges need chunk % kBucketTile == 0)
 // src_bits (nullable): also the TLS guide's RAW-source words (raw_bits then holds its raw words)
 cudaError_t launch_prof_classify(const Job &j, void *ws, const Layout &lo, uint32_t *raw_bits,
                                  int64_t chunk, int64_t *chunk_counts, cudaStream_t st, uint32_t *src_bits = nullptr,

@@ -63,7 +63,8 @@ struct Flow {
   DLoop L;
   const uint32_t *graw, *gsrc;
   unsigned long long *V;
-  uint32_t G, g, n, io;
+  const int32_t *wsrc;   // nullable: writer of each raw iteration's read (loop-local id)
+  uint32_t G, g, n, io, lo;
   uint32_t viol = 0;
   bool lost = false;
 
@@ -84,6 +85,12 @@ struct Flow {
       s.w[k] = L.w ? __ldcs(L.w + i) : (int32_t)(io + i);
       s.gr[k] = __ldcs(graw + (i >> 5));
       s.gs[k] = __ldcs(gsrc + (i >> 5));
+    }
+    if (wsrc) {   // a range of a loop: a raw read written before the range reads A
+#pragma unroll
+      for (int k = 0; k < kFlowK; k++)
+        if (act(base, k) && raw_bit(s, base, k) && (uint32_t)__ldcs(wsrc + it(base, k)) < lo)
+          s.gr[k] &= ~(1u << (it(base, k) & 31));
     }
   }
   // exposed reads of the non-violators (the violators' operands come from V)
@@ -129,9 +136,10 @@ struct Flow {
 
 template <int DT>
 __global__ void __launch_bounds__(kFlowT, JP_FLOW_MINB) k_tls_flow(DLoop L, const uint32_t *graw, const uint32_t *gsrc,
-                                                       unsigned long long *V, int64_t *stats) {
+                                                       unsigned long long *V, int64_t *stats, const int32_t *wsrc,
+                                                       uint32_t lo) {
   Flow<DT> F;
-  F.L = L; F.graw = graw; F.gsrc = gsrc; F.V = V;
+  F.L = L; F.graw = graw; F.gsrc = gsrc; F.V = V; F.wsrc = wsrc; F.lo = lo;
   F.G = gridDim.x * (uint32_t)kFlowT;
   F.g = blockIdx.x * (uint32_t)kFlowT + threadIdx.x;
   F.n = (uint32_t)L.n;
@@ -160,7 +168,7 @@ __global__ void __launch_bounds__(kFlowT, JP_FLOW_MINB) k_tls_flow(DLoop L, cons
 
 template <int DT>
 static cudaError_t run_flow(const Job &j, const uint32_t *graw, const uint32_t *gsrc, unsigned long long *V,
-                            int64_t *stats, cudaStream_t st) {
+                            int64_t *stats, cudaStream_t st, const int32_t *wsrc, uint32_t lo) {
   int maxb = 0;
   cudaOccupancyMaxActiveBlocksPerMultiprocessor(&maxb, (const void *)k_tls_flow<DT>, kFlowT, 0);
   if (maxb < 1) return cudaErrorInvalidConfiguration;
@@ -168,7 +176,7 @@ static cudaError_t run_flow(const Job &j, const uint32_t *graw, const uint32_t *
   const int64_t need = (j.d.n + kFlowT - 1) / kFlowT;
   if (need < grid) grid = (int)(need < 1 ? 1 : need);
   DLoop d = j.d;
-  void *args[] = {&d, &graw, &gsrc, &V, &stats};
+  void *args[] = {&d, &graw, &gsrc, &V, &stats, &wsrc, &lo};
   note_launch();
   return cudaLaunchCooperativeKernel((const void *)k_tls_flow<DT>, dim3(grid), dim3(kFlowT), args, 0, st);
 }
@@ -179,12 +187,12 @@ static cudaError_t run_flow(const Job &j, const uint32_t *graw, const uint32_t *
 // (committed n, executed n + violations, windows 1).  V must hold no value
 // tagged 1 << 32 for an address the loop writes (zeroed).
 cudaError_t launch_tls_flow(const Job &j, const uint32_t *graw, const uint32_t *gsrc, unsigned long long *V,
-                            int64_t *stats, cudaStream_t st) {
+                            int64_t *stats, cudaStream_t st, const int32_t *wsrc, int64_t lo) {
   cudaMemsetAsync(stats, 0, 4 * sizeof(int64_t), st);
   if (j.d.n == 0) return launch_check();
   if (j.op != JP_OP_ADD_C) return cudaErrorInvalidValue;
-  cudaError_t e = j.dt == JP_F32 ? run_flow<JP_F32>(j, graw, gsrc, V, stats, st)
-                                 : run_flow<JP_I32>(j, graw, gsrc, V, stats, st);
+  cudaError_t e = j.dt == JP_F32 ? run_flow<JP_F32>(j, graw, gsrc, V, stats, st, wsrc, (uint32_t)lo)
+                                 : run_flow<JP_I32>(j, graw, gsrc, V, stats, st, wsrc, (uint32_t)lo);
   if (e != cudaSuccess) return e;
   return launch_check();
 }

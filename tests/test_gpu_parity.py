@@ -1052,7 +1052,7 @@ def test_schedule_stealing_two_grid_tls_tasks():
     res = jp.jp_schedule(L, jp.workspace(L), scheme=jp.JP_SCHED_STEALING, chunk_iters=4096)
     torch.cuda.synchronize()
     check_arrays(gw, Aexp, None)
-    assert res["n_tasks"] == 4 and res["task_mode_iters"][jp.JP_MODE_TLS] == 2 * m and res["tls_path"] == 6, res
+    assert res["n_tasks"] == 4 and res["task_mode_iters"][jp.JP_MODE_TLS] == 2 * m and res["tls_path"] in (6, 8), res
 
 
 @pytest.mark.parametrize("full", ["0", "1"])
@@ -1173,3 +1173,31 @@ def test_schedule_bucket_profile_bad_index():
         assert e.value.status == -5
         torch.cuda.synchronize()
         assert torch.equal(g.A, A0)
+
+
+@pytest.mark.parametrize("masks_always", ["0", "1"])
+def test_schedule_stealing_bucket_ranges_dependent(masks_always, monkeypatch):
+    """Large A (the bucket profile) with chunks a multiple of its 16384-iteration
+    tile: the task ranges come from the profile's per-chunk address ranges.  The
+    second half reads what the first half wrote (a cross-task RAW): the PDG must
+    order them; a third, disjoint region overlaps nothing."""
+    if masks_always == "1":
+        monkeypatch.setenv("JP_TASK_MASKS_ALWAYS", "1")
+    q = 1 << 18
+    n = 3 * q
+    ar = torch.arange(n, dtype=torch.int32)
+    g0 = np.random.default_rng(12)
+    w = ar.clone()
+    r = ar.clone()
+    r[q:2 * q] = torch.from_numpy(g0.permutation(q).astype(np.int32))   # reads the first region's writes
+    w[2 * q:] = torch.from_numpy((2 * q + g0.permutation(q)).astype(np.int32))
+    r[2 * q:] = w[2 * q:]
+    wl = synth.Workload("dep_big", O.OP_ADD_C, O.I32, n, torch.from_numpy(g0.integers(0, 99, n + (1 << 20)).astype(np.int32)),
+                        r=r, w=w, c0=5)
+    _, A, _ = O.run_seq(to_oracle(wl))
+    g = gpu(wl)
+    L = jp.Loop.from_workload(g)
+    res = jp.jp_schedule(L, jp.workspace(L), scheme=jp.JP_SCHED_STEALING, chunk_iters=1 << 16)
+    torch.cuda.synchronize()
+    check_arrays(g, A, None)
+    assert res["n_batches"] == 2, res
