@@ -259,17 +259,15 @@ __device__ void merge_p2p_epilogue(const DLoop &L, const unsigned long long *kT,
 // counted into *vbad, nullable) and the per-CTA last-writer table, flushed as
 // packed keys (the value c0*X[i] recomputed at the CTA's last writer of a slot);
 // a grid barrier; then, only if no index was bad, phase 2 streams X into Y =
-// c0*X + c1 and the merged keys reach T -- applied by every CTA (one rank), or,
-// with MERGE, pushed to every rank's inbox by CTA 0 right after the barrier and
-// merged at its end, so the exchange overlaps the Y stream.  s, X and Y each
+// c0*X + c1 and every CTA applies a slice of the keys to T.  s, X and Y each
 // cross HBM once: 12 B/iter, the check included.
 // 4 stages of 32 KiB per phase (the same 128 KiB of shared memory as the one-pass
 // kernel): 16 KiB tiles left each CTA bound by its per-tile barrier / bulk-store
 // turnaround in the X -> Y phase (188 us for config 4, ncu)
 constexpr int kPh = kPrivStages, kPh2Tile = 2 * kPrivTile, kPh2Threads = 1024;
-template <int DT, bool MERGE>
+template <int DT>
 __global__ void __launch_bounds__(kPh2Threads, 1) k_priv_tmp_2ph(DLoop L, unsigned long long *kT, int64_t ntiles,
-                                                                     int64_t *vbad, MergeP2P M) {
+                                                                     int64_t *vbad) {
   extern __shared__ __align__(128) uint32_t psm[];   // [kPh][tile] then tT[lenT]
   __shared__ __align__(8) unsigned long long full1[kPh], full2[kPh];
   uint32_t *tT = psm + (size_t)kPh * kPh2Tile;
@@ -338,14 +336,9 @@ __global__ void __launch_bounds__(kPh2Threads, 1) k_priv_tmp_2ph(DLoop L, unsign
   }
   cg::this_grid().sync();   // every CTA's keys are in, every index checked
   if (vbad && *reinterpret_cast<volatile int64_t *>(vbad)) return;   // nothing written (reading A13)
-  MergeState ms{};
-  if constexpr (MERGE) {
-    if (blockIdx.x == 0) ms = merge_p2p_push(L, kT, M);
-  } else {
-    for (int64_t b = (int64_t)blockIdx.x * kPh2Threads + tid; b < L.lenT; b += (int64_t)gridDim.x * kPh2Threads) {
-      const unsigned long long key = __ldcg(&kT[b]);
-      if (key) L.T[b] = (uint32_t)key;
-    }
+  for (int64_t b = (int64_t)blockIdx.x * kPh2Threads + tid; b < L.lenT; b += (int64_t)gridDim.x * kPh2Threads) {
+    const unsigned long long key = __ldcg(&kT[b]);
+    if (key) L.T[b] = (uint32_t)key;
   }
   // ---------------- phase 2: X -> Y ----------------
   auto issue2 = [&](int64_t k) {
@@ -383,17 +376,14 @@ __global__ void __launch_bounds__(kPh2Threads, 1) k_priv_tmp_2ph(DLoop L, unsign
   if (blockIdx.x == 0)
     for (int64_t i = ntiles * kPh2Tile + tid; i < L.n; i += kPh2Threads)
       L.A[i] = op_add<DT>(op_mul<DT>(L.c0, L.X[i]), L.c1);
-  if constexpr (MERGE) {
-    if (blockIdx.x == 0) merge_p2p_finish(L, M, ms);
-  }
 }
 
 // fuse_apply (cooperative launch): after every CTA's flush a grid barrier, then
 // the keys are applied to T by every CTA (R1 + R2 in one launch when the index
 // check is not needed; k_priv_tmp_2ph carries the check)
-template <int DT>
+template <int DT, bool MERGE = false>
 __global__ void __launch_bounds__(kPrivTmaThreads, 1) k_priv_tmp_tma(DLoop L, unsigned long long *kT, int64_t ntiles,
-                                                                     int fuse_apply) {
+                                                                     int fuse_apply, MergeP2P M = MergeP2P{}) {
   if (aborted(L)) return;
   extern __shared__ __align__(128) uint32_t psm[];   // [stage][2][tile] then tT[lenT]
   __shared__ __align__(8) unsigned long long full[kPrivStages];
@@ -467,6 +457,10 @@ __global__ void __launch_bounds__(kPrivTmaThreads, 1) k_priv_tmp_tma(DLoop L, un
   }
   if (fuse_apply) {
     cg::this_grid().sync();   // every CTA's keys are in
+    if constexpr (MERGE) {   // C4 across the ranks and R2, by CTA 0 (jp_priv_stream_merge)
+      if (blockIdx.x == 0) merge_p2p_epilogue(L, kT, M);
+      return;
+    }
     for (int64_t b = (int64_t)blockIdx.x * kPrivTmaThreads + tid; b < L.lenT; b += (int64_t)gridDim.x * kPrivTmaThreads) {
       const unsigned long long k = __ldcg(&kT[b]);
       if (k) L.T[b] = (uint32_t)k;
@@ -519,7 +513,8 @@ static void run_priv(const DLoop &d0, unsigned long long *kA, unsigned long long
           DLoop dd = d;
           int64_t nt = ntiles;
           int fuse = 1;
-          void *args[] = {&dd, &kT, &nt, &fuse};
+          MergeP2P none{};
+          void *args[] = {&dd, &kT, &nt, &fuse, &none};
           cudaLaunchCooperativeKernel((void *)k_priv_tmp_tma<DT>, dim3(g), dim3(kPrivTmaThreads), args, smem, st);
           *applied = true;
         } else if (fuse_apply) {   // with the index check: two phases (s, then X -> Y)
@@ -534,14 +529,13 @@ static void run_priv(const DLoop &d0, unsigned long long *kA, unsigned long long
           int64_t nt = ntiles;
           int64_t *vb = vbad;
           if (vb) cudaMemsetAsync(vb, 0, sizeof(int64_t), st);
-          MergeP2P none{};
-          void *args[] = {&dd, &kT, &nt, &vb, &none};
-          cudaFuncSetAttribute(k_priv_tmp_2ph<DT, false>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-          cudaLaunchCooperativeKernel((void *)k_priv_tmp_2ph<DT, false>, dim3(g), dim3(kPh2Threads), args, smem, st);
+          void *args[] = {&dd, &kT, &nt, &vb};
+          cudaFuncSetAttribute(k_priv_tmp_2ph<DT>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+          cudaLaunchCooperativeKernel((void *)k_priv_tmp_2ph<DT>, dim3(g), dim3(kPh2Threads), args, smem, st);
           *applied = true;
         } else {
           validate_first();
-          k_priv_tmp_tma<DT><<<g, kPrivTmaThreads, smem, st>>>(d, kT, ntiles, 0);
+          k_priv_tmp_tma<DT><<<g, kPrivTmaThreads, smem, st>>>(d, kT, ntiles, 0, MergeP2P{});
         }
         note_launch();
         return;
@@ -582,8 +576,12 @@ cudaError_t launch_priv_stream_merge(const Job &j, unsigned long long *kT, unsig
   d.A += d.ioff; d.lenA -= d.ioff;
   d.ioff = 0;
   cudaMemsetAsync(kT, 0, 8 * (size_t)d.lenT, st);
-  const int64_t ntiles = d.n / kPh2Tile;
-  const size_t smem = (size_t)kPh * kPh2Tile * 4 + (size_t)d.lenT * 4;
+  // the one-pass stream (the ranks' indices were checked by the partitioned
+  // profile) with the merge as its epilogue: measured faster than merging from
+  // the two-phase kernel, whose s-only phase costs more than the overlap of the
+  // exchange with the Y stream saves
+  const int64_t ntiles = d.n / kPrivTile;
+  const size_t smem = (size_t)kPrivStages * 2 * kPrivTile * 4 + (size_t)d.lenT * 4;
   cudaError_t e;
   auto go = [&](auto kern) {
     cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
@@ -595,12 +593,12 @@ cudaError_t launch_priv_stream_merge(const Job &j, unsigned long long *kT, unsig
     M.me = me;
     M.err = err;
     int64_t nt = ntiles;
-    int64_t *vb = nullptr;   // (the ranks' indices were checked by the partitioned profile)
-    void *args[] = {&d, &kT, &nt, &vb, &M};
-    e = cudaLaunchCooperativeKernel((const void *)kern, dim3(g), dim3(kPh2Threads), args, smem, st);
+    int fuse = 1;
+    void *args[] = {&d, &kT, &nt, &fuse, &M};
+    e = cudaLaunchCooperativeKernel((const void *)kern, dim3(g), dim3(kPrivTmaThreads), args, smem, st);
   };
-  if (j.dt == JP_F32) go(k_priv_tmp_2ph<JP_F32, true>);
-  else go(k_priv_tmp_2ph<JP_I32, true>);
+  if (j.dt == JP_F32) go(k_priv_tmp_tma<JP_F32, true>);
+  else go(k_priv_tmp_tma<JP_I32, true>);
   note_launch();
   if (e != cudaSuccess) return e;
   return launch_check();
