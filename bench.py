@@ -685,10 +685,24 @@ def partitioned_config5(jp, dev, st, world, rank, steps):
         barrier(world)
         if k >= 2:
             ts.append(time.perf_counter() - t0)
-    # one more call with per-phase CUDA events (not in the timing above)
+    # one more call with per-phase CUDA events (not in the timing above); at one
+    # rank the driver runs jp_schedule(STEALING): the multi-rank path itself is
+    # timed too (force_ranks), with its phases
     wl.A.copy_(A0)
     barrier(world)
-    ph = jd.schedule_stealing(full, ws, chunk_iters=65536, timings=True)["phases"]
+    ph = jd.schedule_stealing(full, ws, chunk_iters=65536, timings=True, force_ranks=True)["phases"]
+    forced_ms = None
+    if world == 1:
+        fts = []
+        for k in range(6):
+            wl.A.copy_(A0)
+            torch.cuda.synchronize()
+            t0 = time.perf_counter()
+            jd.schedule_stealing(full, ws, chunk_iters=65536, force_ranks=True)
+            torch.cuda.synchronize()
+            if k >= 1:
+                fts.append(time.perf_counter() - t0)
+        forced_ms = statistics.median(fts) * 1e3
     # device-side stealing (jp_run_priv_claim): chunks claimed at run time
     dts, dres = [], {"rank_work": "skipped: CUDA-IPC rows turned off (JP_BENCH_IPC=0)"}
     try:
@@ -719,7 +733,8 @@ def partitioned_config5(jp, dev, st, world, rank, steps):
     out = {"workload": "config5 mixed ADD_C int32 N=2^24, multi-rank task stealing (chunk 2^16)", "ms": ms,
            "iters_per_s": wl.n / (ms * 1e-3), "n_tasks": res["n_tasks"], "n_batches": res["n_batches"],
            "rank0_iters": res["rank_work"]["iters"], "tls": res["tls"], "phases_max_over_ranks": phases,
-           "busy_ms_per_rank": busy, "stolen_chunks": n_stolen,
+           "busy_ms_per_rank": busy, "stolen_chunks": n_stolen, "multi_rank_path_ms_at_one_rank": forced_ms,
+           "delegated": res.get("delegated"),
            "dynamic": {"ms": dyn_ms, "iters_per_s": wl.n / (dyn_ms * 1e-3) if dyn_ms else None,
                        "rank0": dres["rank_work"],
                        "what": "the batch's partitioned chunks claimed on the device (jp_run_priv_claim)"},

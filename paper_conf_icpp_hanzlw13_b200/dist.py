@@ -393,7 +393,7 @@ def _levels(conf, nt):
 
 def schedule_stealing(full, ws, group=None, chunk_iters: int = 65536, tau_high: float = _abi.TAU_HIGH, speed=None,
                       speed_tls: float = 1.0, exchange: str = "dense", engine=None, timings: bool = False,
-                      dynamic: bool = False) -> dict:
+                      dynamic: bool = False, force_ranks: bool = False) -> dict:
     """Task stealing of one loop across the ranks (Alg. 1; SURVEY
     Sec.8(e) "Mixed").  Every rank holds full replicas (``full``, workspace
     ``ws`` of the whole loop):
@@ -420,10 +420,30 @@ def schedule_stealing(full, ws, group=None, chunk_iters: int = 65536, tau_high: 
          through identity indices (no key table, e.g. config 4's Y) stay with
          the rank that executed the chunk, as under task sharing (``chunks``
          of the result gives the owners).
+
+    A one-rank group has nothing to exchange: it runs the single-GPU
+    scheduler, jp_schedule(STEALING) -- the same Alg. 1 plan without the
+    partitioned profile, the key exchange and the privatized replicas
+    (``force_ranks=True`` keeps the multi-rank path, e.g. to measure it).
     """
     jp = _engine(engine)
     world, rank = world_rank(group)
     n = full.n
+    if world == 1 and not dynamic and not force_ranks and hasattr(jp, "jp_schedule"):
+        ev = [torch.cuda.Event(enable_timing=True) for _ in range(2)] if timings else None
+        if ev:
+            ev[0].record()
+        res = jp.jp_schedule(full, ws, scheme=_abi.JP_SCHED_STEALING, chunk_iters=chunk_iters, tau_high=tau_high)
+        phases = None
+        if ev:
+            ev[1].record()
+            torch.cuda.synchronize()
+            phases = {"profile_ms": 0.0, "plan_ms": 0.0, "busy_ms": ev[0].elapsed_time(ev[1]), "merge_ms": 0.0,
+                      "what": "one rank: jp_schedule(STEALING), phases not separated"}
+        return {"scheme": "stealing", "phases": phases, "prof": res["prof"], "n_tasks": res["n_tasks"],
+                "n_batches": res["n_batches"], "tasks": None, "chunks": [(0, n, res["mode"], 0)], "stolen": 0,
+                "tls": res["tls"], "rank_work": {"chunks": -(-n // chunk_iters), "iters": n},
+                "delegated": "jp_schedule(STEALING)"}
     nck = -(-n // chunk_iters)
     marks = []   # (phase, event) on the current stream when timings=True
 

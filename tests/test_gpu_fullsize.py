@@ -84,15 +84,17 @@ def test_config5_full_size_schedule(recovery):
         assert res["tls"] == O.sim_tls(mid, 0, res["tls_w_max"], O.profile(mid)["raw_iters"])[3]
 
 
-@pytest.mark.parametrize("dynamic", [False, True])
-def test_config5_full_size_dist_world1(dynamic):
+@pytest.mark.parametrize("dynamic,force", [(False, False), (False, True), (True, False)])
+def test_config5_full_size_dist_world1(dynamic, force):
     """Config 5 at N = 2^24 through the multi-rank stealing driver at world 1
-    (the bench's partitioned row): every byte of A."""
+    (the bench's partitioned row; force: the multi-rank path instead of the
+    one-rank delegation to jp_schedule): every byte of A."""
     wl = synth.config5()
     ref = to_oracle(wl)
     g = wl.to(DEV)
     L = jp.Loop.from_workload(g)
-    res = jd.schedule_stealing(L, jp.workspace(L), chunk_iters=1 << 16, dynamic=dynamic)
+    res = jd.schedule_stealing(L, jp.workspace(L), chunk_iters=1 << 16, dynamic=dynamic, force_ranks=force)
+    assert ("delegated" in res) == (not dynamic and not force)
     torch.cuda.synchronize()
     _, A, _ = O.run_seq(ref)
     assert equal_bytes(g.A, A), first_diff(g.A, A)
