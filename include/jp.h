@@ -120,11 +120,18 @@ typedef struct { int64_t committed, executed, windows, violations; } jp_tls_stat
  *   cluster, W <= 2048*cluster, cluster 1..16 (0 = auto: the smallest power of
  *   two that holds W, or n when W = 0); 6 every SM (cooperative), W <= 3072 *
  *   co-resident CTAs (454656 on a 148-SM B200, jp_tls_grid_window), write log and shadow values in
- *   workspace regions 7 and 8 (JP_WS_TLS); 0 = auto (5 when W, or n if W = 0,
- *   fits a 16-CTA cluster, else 6).  w_max is ignored.  stats: windows, violations =
- *   violating iterations, executed = n + violations, committed = n.  A second
- *   writer of an address found at run time (a wrong profile) gives JP_ERR_ARG
- *   after the run, with A in an unspecified state.                          */
+ *   workspace regions 7 and 8 (JP_WS_TLS); 8 ONE window of the whole loop
+ *   (reading B12; W must be 0 or >= n): ADD_C only, a profile with war_iters ==
+ *   waw_iters == 0 and guided = 1 (the guide words of that profile, from
+ *   jp_tls_guide or jp_schedule) -- the violators are the guide's raw
+ *   iterations, non-violators commit in place at once, violators wait for their
+ *   writer's shadow slot (region 8, JP_WS_TLS); no write log, no barrier;
+ *   0 = auto (5 when W, or n if W = 0, fits a 16-CTA cluster, else 6; jp_schedule
+ *   picks 8 itself when it applies).  w_max is ignored.  stats: windows,
+ *   violations = violating iterations, executed = n + violations, committed =
+ *   n.  A second writer of an address found at run time (a wrong profile) gives
+ *   JP_ERR_ARG after the run, with A in an unspecified state (path 8: a
+ *   violator whose writer never published, after a ~seconds-long wait).     */
 typedef enum { JP_TLS_RESTART = 0, JP_TLS_ONCHIP = 1 } jp_tls_recovery;
 typedef struct {
   int64_t window; int64_t w_max; int32_t path; int32_t cluster;
@@ -171,10 +178,10 @@ typedef struct {
   int32_t tls_path;             /* TLS: jp_tls_cfg.path that ran (1, 2, 3; 4 tiny
                                    one-CTA schedule; 5 / 6 on-chip recovery on a
                                    cluster / on every SM; 7 one-warp program order
-                                   for mode C)                                    */
+                                   for mode C; 8 on-chip recovery in one window)  */
   int32_t tls_guided;           /* TLS: 1 when the guide (jp_tls_guide) steered it    */
   int32_t tls_recovery;         /* TLS: jp_tls_recovery that ran                      */
-  int32_t tls_cluster;          /* TLS: CTAs of the cluster (paths 3, 5) or grid (6)  */
+  int32_t tls_cluster;          /* TLS: CTAs of the cluster (paths 3, 5) or grid (6, 8) */
 } jp_sched_result;
 
 /* ---- workspace -------------------------------------------------------------
