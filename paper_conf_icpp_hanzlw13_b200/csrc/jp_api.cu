@@ -1736,7 +1736,10 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
   // stream from the start, overlapping the static check's prefix read
   const Layout lg = layout(L);
   const bool gfuse = lg.bytes[R_GUIDE] && ws && ws_bytes >= layout_end(lg, JP_WS_PROFILE | JP_WS_GUIDE | JP_WS_TLS);
-  const bool pairs = gfuse && stamp_pairs_ok(j, ws, lg);
+  // the address-bucket profile keeps no tables: no pair table to pre-fill (the
+  // TLS paths that use region 7 reset it themselves)
+  const bool bucket = gfuse && bucket_profile_ok(j, ws, lg);
+  const bool pairs = gfuse && !bucket && stamp_pairs_ok(j, ws, lg);
   cudaEvent_t pdone = nullptr;
   if (pairs && cudaEventCreateWithFlags(&pdone, cudaEventDisableTiming) == cudaSuccess) {
     cudaStream_t side = g_pool.get(41);
@@ -1793,7 +1796,7 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
     // the on-chip TLS shadow values must start at zero: clear them on a side
     // stream while the (L2-atomic-bound) profile runs, instead of after it
     auto *V = at<unsigned long long>(ws, lg, R_TLS_C_A);
-    if (pairs && V && cudaEventCreateWithFlags(&vdone, cudaEventDisableTiming) == cudaSuccess) {
+    if ((pairs || bucket) && V && cudaEventCreateWithFlags(&vdone, cudaEventDisableTiming) == cudaSuccess) {
       cudaStream_t side = g_pool.get(40);
       cudaEventRecord(vdone, st);          // after whatever ran before on st
       cudaStreamWaitEvent(side, vdone, 0);
@@ -1802,7 +1805,7 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
       clean = 2;
     }
     if (pairs) clean |= 1;   // region 7 holds this call's pair table, or the side stream's all-ones fill
-    if (bucket_profile_ok(j, ws, lg)) {
+    if (bucket) {
       // large A: the profile by address buckets (jp_bucket.cu), guide words included
       uint32_t *g = at<uint32_t>(ws, lg, R_GUIDE);
       JP_CUDA(launch_prof_bucket(j, ws, lg, g, g + (L->n + 31) / 32, 0, nullptr, st), "profile (buckets)");
