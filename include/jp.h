@@ -332,7 +332,11 @@ jp_status jp_run_tls(const jp_loop *L, const jp_tls_cfg *cfg /* host */, const j
  * recovery.  The workspace is scratch for the whole call: the profile tables
  * of large loops are kept interleaved in the TLS region and the minW / minR
  * regions are not left filled (call jp_profile_density for the tables).
- * syncs.                                                                     */
+ * syncs until res is complete (the mode, the profile, the index check); the
+ * loop's last writes may still be running on st when it returns (the
+ * structurally RAW-free privatized run returns after its index check, before
+ * its X -> Y phase; a DOALL exit does not wait at all): read the arrays after
+ * st, as for any stream-ordered call.                                      */
 jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfg /* host */, void *ws,
                       size_t ws_bytes, jp_sched_result *res /* host */, jp_stream_t st);
 /* Same, with every array pointer of L_host on the HOST (pinned for speed): the

@@ -1713,16 +1713,37 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
       int64_t *bad = &at<int64_t>(ws, lo, R_HEADER)[H_BAD];
       Job jr = j;
       jr.d.abort = bad;
+      int64_t nb = 0;
+      bool published = false;
       if (smode == JP_MODE_PRIVATIZED) {
+        // the two-phase kernel publishes its index count to mapped host words
+        // (tiny mirror [17] count, [18] sequence) when its check is done: the
+        // call returns then, the X -> Y phase runs on, ordered on st
+        TinyMirror &m = tiny_mirror();
+        const bool mir = m.host && !getenv("JP_STRUCT_NO_MIRROR");
+        const unsigned long long seq = mir ? ++m.seq : 0;
         bool applied = false;
-        JP_CUDA(launch_priv_stream(jr, ws, lo, true, st, 0, true, &applied, bad), "priv stream");
+        JP_CUDA(launch_priv_stream(jr, ws, lo, true, st, 0, true, &applied, bad, mir ? m.dev + 17 : nullptr, seq,
+                                   &published),
+                "priv stream");
         if (!applied) JP_CUDA(launch_priv_finalize(jr, ws, lo, st), "priv finalize");
+        if (published) {
+          volatile unsigned long long *flag = reinterpret_cast<volatile unsigned long long *>(&m.host[18]);
+          for (unsigned spins = 0; *flag != seq; spins++) {
+            if ((spins & 1023) == 1023) {
+              const cudaError_t q = cudaStreamQuery(st);
+              if (q != cudaSuccess && q != cudaErrorNotReady) return cuda_fail(q, "priv stream");
+              if (q == cudaSuccess && *flag != seq)
+                return fail(JP_ERR_CUDA, "privatized kernel finished without publishing its index check");
+            }
+          }
+          nb = *reinterpret_cast<volatile int64_t *>(&m.host[17]);
+        }
       } else {
         JP_CUDA(launch_validate_indirect(j, bad, st), "validate");
         JP_CUDA(launch_doall(jr, st), "doall");
       }
-      int64_t nb = 0;
-      JP_CUDA(d2h_small_sync(&nb, bad, sizeof nb, st), "validate D2H");
+      if (!published) JP_CUDA(d2h_small_sync(&nb, bad, sizeof nb, st), "validate D2H");
       if (nb) return fail(JP_ERR_INDEX, "%lld index entries are outside their arrays", (long long)nb);
       res->mode = smode;
       res->profiled = 0;

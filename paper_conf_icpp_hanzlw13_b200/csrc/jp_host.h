@@ -94,9 +94,13 @@ void set_doall_kernel_choice(int v);
 // validate (nullable): count out-of-range indirect indices into *validate before
 // anything is written (reading A13; j.d.abort should point at it so that every
 // later kernel of the run exits when it is nonzero)
+// mirror (nullable, mapped host words): the two-phase kernel (fused apply with
+// validate) writes mirror[0] = the count, then mirror[1] = seq, as soon as the
+// check is done; *published tells whether that kernel ran (else read *validate)
 cudaError_t launch_priv_stream(const Job &j, void *ws, const Layout &lo, bool clear_keys,
                                cudaStream_t st, int max_ctas = 0, bool fuse_apply = false, bool *applied = nullptr,
-                               int64_t *validate = nullptr);
+                               int64_t *validate = nullptr, int64_t *mirror = nullptr, unsigned long long seq = 0,
+                               bool *published = nullptr);
 cudaError_t launch_priv_finalize(const Job &j, void *ws, const Layout &lo, cudaStream_t st);
 cudaError_t launch_merge_apply(void *arr, int64_t len, const int64_t *keys, cudaStream_t st);
 // mode C on the device (jp_serial.cu): one warp runs the loop in program order; stats[4] as TLS

@@ -18,6 +18,7 @@
 // flush then recomputes the winner's value and issues one 64-bit global
 // atomicMax per (CTA, touched slot).
 #include <cooperative_groups.h>
+#include <atomic>
 #include <cstring>
 #include "jp_host.h"
 
@@ -267,13 +268,20 @@ __device__ void merge_p2p_epilogue(const DLoop &L, const unsigned long long *kT,
 constexpr int kPh = kPrivStages, kPh2Tile = 2 * kPrivTile, kPh2Threads = 1024;
 template <int DT>
 __global__ void __launch_bounds__(kPh2Threads, 1) k_priv_tmp_2ph(DLoop L, unsigned long long *kT, int64_t ntiles,
-                                                                     int64_t *vbad) {
+                                                                     int64_t *vbad, int64_t *mirror,
+                                                                     unsigned long long seq) {
   extern __shared__ __align__(128) uint32_t psm[];   // [kPh][tile] then tT[lenT]
   __shared__ __align__(8) unsigned long long full1[kPh], full2[kPh];
   uint32_t *tT = psm + (size_t)kPh * kPh2Tile;
   const int tid = threadIdx.x;
   const uint32_t lenT = (uint32_t)L.lenT;
   for (int64_t k = tid; k < L.lenT; k += kPh2Threads) tT[k] = 0;
+  // the key table and the index-error count are cleared here (no memset
+  // launches ahead of the kernel); the grid barrier after phase 1 orders the
+  // clears before every CTA's flush
+  for (int64_t b = (int64_t)blockIdx.x * kPh2Threads + tid; b < L.lenT; b += (int64_t)gridDim.x * kPh2Threads)
+    kT[b] = 0;
+  if (vbad && blockIdx.x == 0 && tid == 0) *vbad = 0;
   const int64_t my = ntiles > blockIdx.x ? (ntiles - 1 - blockIdx.x) / gridDim.x + 1 : 0;
   auto tile_of = [&](int64_t k) { return ntiles - 1 - (int64_t)blockIdx.x - k * gridDim.x; };
   auto buf = [&](int64_t k) { return psm + (size_t)(k % kPh) * kPh2Tile; };
@@ -328,14 +336,21 @@ __global__ void __launch_bounds__(kPh2Threads, 1) k_priv_tmp_2ph(DLoop L, unsign
       if ((uint32_t)sv < lenT) smem_last(tT, sv, i); else bad++;
     }
   bad = __reduce_add_sync(0xffffffffu, bad);
+  cg::this_grid().sync();   // the clears above are visible to every CTA
   if (vbad && (tid & 31) == 0 && bad) atomicAdd(reinterpret_cast<unsigned long long *>(vbad), (unsigned long long)bad);
-  __syncthreads();
   for (int64_t b = tid; b < L.lenT; b += kPh2Threads) {
     const uint32_t e = tT[b];
     if (e) atomicMax(&kT[b], pack_key(L.base + e - 1, op_mul<DT>(L.c0, __ldg(L.X + e - 1))));
   }
   cg::this_grid().sync();   // every CTA's keys are in, every index checked
-  if (vbad && *reinterpret_cast<volatile int64_t *>(vbad)) return;   // nothing written (reading A13)
+  const int64_t nbad = vbad ? *reinterpret_cast<volatile int64_t *>(vbad) : 0;
+  if (mirror && blockIdx.x == 0 && tid == 0) {
+    // the count to mapped host memory, then the call's sequence number: the
+    // host returns as soon as it sees it (the X -> Y phase is stream-ordered)
+    mirror[0] = nbad;
+    asm volatile("st.release.sys.global.u64 [%0], %1;" ::"l"(mirror + 1), "l"(seq) : "memory");
+  }
+  if (nbad) return;   // nothing written (reading A13)
   for (int64_t b = (int64_t)blockIdx.x * kPh2Threads + tid; b < L.lenT; b += (int64_t)gridDim.x * kPh2Threads) {
     const unsigned long long key = __ldcg(&kT[b]);
     if (key) L.T[b] = (uint32_t)key;
@@ -481,7 +496,15 @@ static bool al16(const void *p) { return ((uintptr_t)p & 15) == 0; }
 
 template <int OP, int DT>
 static void run_priv(const DLoop &d0, unsigned long long *kA, unsigned long long *kT, cudaStream_t st, int max_ctas,
-                     bool fuse_apply, bool *applied, int64_t *vbad) {
+                     bool fuse_apply, bool *applied, int64_t *vbad, bool clear_keys, int64_t *mirror,
+                     unsigned long long seq, bool *published) {
+  // the key tables start at zero: cleared here, except by the two-phase kernel
+  // (which clears its table itself)
+  auto clear = [&]() {
+    if (!clear_keys) return;
+    if (kA) cudaMemsetAsync(kA, 0, 8 * (size_t)d0.lenA, st);
+    if (kT) cudaMemsetAsync(kT, 0, 8 * (size_t)d0.lenT, st);
+  };
   // vbad: validate the indirect indices first (reading A13), one streaming pass
   // ahead of the run (an in-kernel phase before a grid barrier was measured
   // slower: 177 vs ~169 us device time on config 4); the stream kernels then
@@ -510,6 +533,7 @@ static void run_priv(const DLoop &d0, unsigned long long *kA, unsigned long long
         if (max_ctas > 0 && g > max_ctas) g = max_ctas;
         if (ntiles < g) g = (int)(ntiles < 1 ? 1 : ntiles);
         if (fuse_apply && !vbad) {   // R1 + R2 in one pass (cooperative: one CTA per SM, co-resident)
+          clear();
           DLoop dd = d;
           int64_t nt = ntiles;
           int fuse = 1;
@@ -528,12 +552,25 @@ static void run_priv(const DLoop &d0, unsigned long long *kA, unsigned long long
           dd.abort = nullptr;
           int64_t nt = ntiles;
           int64_t *vb = vbad;
-          if (vb) cudaMemsetAsync(vb, 0, sizeof(int64_t), st);
-          void *args[] = {&dd, &kT, &nt, &vb};
-          cudaFuncSetAttribute(k_priv_tmp_2ph<DT>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+          int64_t *mir = mirror;
+          unsigned long long sq = seq;
+          void *args[] = {&dd, &kT, &nt, &vb, &mir, &sq};
+          // one dynamic-smem limit for every call (lenT <= kSmemSlots), set once per device
+          static std::atomic<unsigned long long> attr{0};
+          int dev = 0;
+          cudaGetDevice(&dev);
+          const unsigned long long bit = 1ull << (dev & 63);
+          if (!(attr.load() & bit)) {
+            const size_t smax = (size_t)kPh * kPh2Tile * 4 + (size_t)kSmemSlots * 4;
+            if (cudaFuncSetAttribute(k_priv_tmp_2ph<DT>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smax) ==
+                cudaSuccess)
+              attr.fetch_or(bit);
+          }
           cudaLaunchCooperativeKernel((void *)k_priv_tmp_2ph<DT>, dim3(g), dim3(kPh2Threads), args, smem, st);
           *applied = true;
+          if (published) *published = mirror != nullptr;
         } else {
+          clear();
           validate_first();
           k_priv_tmp_tma<DT><<<g, kPrivTmaThreads, smem, st>>>(d, kT, ntiles, 0, MergeP2P{});
         }
@@ -543,6 +580,7 @@ static void run_priv(const DLoop &d0, unsigned long long *kA, unsigned long long
       int64_t nvec = d.n / 4;
       int64_t need = (nvec + kPrivThreads * 2 - 1) / (kPrivThreads * 2);
       if (need < grid) grid = (int)(need < 1 ? 1 : need);
+      clear();
       validate_first();
       k_priv_tmp_vec<DT><<<grid, kPrivThreads, d.lenT * 4, st>>>(d, kT, nvec);
       note_launch();
@@ -554,6 +592,7 @@ static void run_priv(const DLoop &d0, unsigned long long *kA, unsigned long long
   size_t smem = ((smA ? d.lenA : 0) + (smT ? d.lenT : 0)) * 4;
   int64_t need = (d.n + kPrivThreads - 1) / kPrivThreads;
   if (need < grid) grid = (int)(need < 1 ? 1 : need);
+  clear();
   validate_first();
   k_priv_generic<OP, DT><<<grid, kPrivThreads, smem, st>>>(d, kA, kT, smA, smT);
   note_launch();
@@ -605,21 +644,25 @@ cudaError_t launch_priv_stream_merge(const Job &j, unsigned long long *kT, unsig
 }
 
 cudaError_t launch_priv_stream(const Job &j, void *ws, const Layout &lo, bool clear_keys, cudaStream_t st,
-                               int max_ctas, bool fuse_apply, bool *applied, int64_t *validate) {
-  bool dummy = false;
+                               int max_ctas, bool fuse_apply, bool *applied, int64_t *validate, int64_t *mirror,
+                               unsigned long long seq, bool *published) {
+  bool dummy = false, dummy2 = false;
   if (!applied) applied = &dummy;
+  if (!published) published = &dummy2;
   *applied = false;
+  *published = false;
   auto *kA = at<unsigned long long>(ws, lo, R_KEYS_A);
   auto *kT = at<unsigned long long>(ws, lo, R_KEYS_T);
-  if (clear_keys) {
-    if (kA) cudaMemsetAsync(kA, 0, lo.bytes[R_KEYS_A], st);
-    if (kT) cudaMemsetAsync(kT, 0, lo.bytes[R_KEYS_T], st);
-  }
   if (j.d.n == 0) {
+    if (clear_keys) {
+      if (kA) cudaMemsetAsync(kA, 0, lo.bytes[R_KEYS_A], st);
+      if (kT) cudaMemsetAsync(kT, 0, lo.bytes[R_KEYS_T], st);
+    }
     if (validate) cudaMemsetAsync(validate, 0, sizeof(int64_t), st);
     return launch_check();
   }
-  JP_DISPATCH(j.op, j.dt, run_priv, j.d, kA, kT, st, max_ctas, fuse_apply, applied, validate);
+  JP_DISPATCH(j.op, j.dt, run_priv, j.d, kA, kT, st, max_ctas, fuse_apply, applied, validate, clear_keys, mirror, seq,
+              published);
   return launch_check();
 }
 

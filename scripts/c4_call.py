@@ -21,3 +21,12 @@ _, ms_run = bench.median_timed(lambda: jp.jp_run_privatized(L, prof, ws, stream=
 hbm, _ = bench.peaks()
 print(f"config4 jp_schedule {ms:.4f} ms ({12 * wl.n / ms / 1e6 / hbm:.3f} of HBM), run alone {ms_run:.4f} ms, "
       f"mode {res['mode_name']} profiled {res['profiled']}")
+torch.cuda.synchronize()
+a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+a.record(st)
+for _ in range(20):
+    jp.jp_schedule(L, ws, stream=st)
+b.record(st)
+torch.cuda.synchronize()
+mp = a.elapsed_time(b) / 20
+print(f"config4 jp_schedule back to back: {mp:.4f} ms per call ({12 * wl.n / mp / 1e6 / hbm:.3f} of HBM)")

@@ -198,6 +198,14 @@ def test_structural_raw_free_schedule(case, doall_kernel):
     assert e.value.status == -5
     torch.cuda.synchronize()
     assert torch.equal(g.A, A0) and (T0 is None or torch.equal(g.T, T0))
+    # a good call on the same workspace right after the aborted one (whose
+    # keys were flushed before the abort): the run clears what it uses
+    g = gpu(wl)
+    L = jp.Loop.from_workload(g)
+    res = jp.jp_schedule(L, ws)
+    torch.cuda.synchronize()
+    assert res["mode"] == mode and res["profiled"] == 0, res
+    check_arrays(g, A, T)
     # static_check = 1: the profile decides (Fig. 2(b)), same arrays
     g = gpu(wl)
     L = jp.Loop.from_workload(g)
@@ -205,6 +213,40 @@ def test_structural_raw_free_schedule(case, doall_kernel):
     torch.cuda.synchronize()
     assert res["profiled"] == 1 and res["prof"]["raw_iters"] == 0
     check_arrays(g, A, T)
+
+
+@pytest.mark.parametrize("mirror", [1, 0])
+def test_structural_priv_side_stream(mirror, monkeypatch):
+    """The structural privatized call returns once its index check is published
+    (mapped host words; JP_STRUCT_NO_MIRROR=1: a device-to-host copy): the
+    X -> Y phase is ordered on the caller's stream, so the arrays equal the
+    oracle after that stream -- back-to-back calls on one workspace with
+    different inputs, one of them with a bad index in between."""
+    if not mirror:
+        monkeypatch.setenv("JP_STRUCT_NO_MIRROR", "1")
+    st = torch.cuda.Stream()
+    ws = None
+    for k in range(4):
+        wl = synth.config4(n=(1 << 19) + 13 * k, slots=(1024, 256, 4096, 512)[k])
+        _, A, T = O.run_seq(to_oracle(wl))
+        g = gpu(wl)
+        torch.cuda.synchronize()
+        L = jp.Loop.from_workload(g)
+        ws = jp.workspace(L) if ws is None or ws.numel() < jp.workspace(L).numel() else ws
+        if k == 2:
+            g.s[7] = -1
+            A0 = g.A.clone()
+            torch.cuda.synchronize()
+            with pytest.raises(jp.JPError) as e:
+                jp.jp_schedule(L, ws, stream=st)
+            assert e.value.status == -5
+            st.synchronize()
+            assert torch.equal(g.A, A0)
+            continue
+        res = jp.jp_schedule(L, ws, stream=st)
+        st.synchronize()
+        assert res["mode"] == jp.JP_MODE_PRIVATIZED and res["profiled"] == 0, res
+        check_arrays(g, A, T)
 
 
 def test_illegal_modes_and_workspace():
