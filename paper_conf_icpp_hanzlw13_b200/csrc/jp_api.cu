@@ -8,6 +8,7 @@
 #include <cstdarg>
 #include <cstdio>
 #include <cstring>
+#include <functional>
 #include <mutex>
 #include <string>
 #include <vector>
@@ -366,6 +367,16 @@ jp_status jp_profile_density(const jp_loop *L, void *ws, size_t ws_bytes, uint32
   return jp_profile_classify(L, ws, ws_bytes, raw_bits, chunk_iters, chunk_counts, out, st);
 }
 
+// the largest raw count whose density is not above tau (select_mode_counts: mode B, not C)
+static int64_t raw_max_for(int64_t n, double tau) {
+  if (n <= 0) return 0;
+  int64_t r = (int64_t)std::floor(tau * (double)n);
+  if (r > n) r = n;
+  while (r + 1 <= n && (double)(r + 1) / (double)n <= tau) r++;
+  while (r >= 0 && (double)r / (double)n > tau) r--;
+  return r;
+}
+
 static int32_t select_mode_counts(int64_t n, int64_t raw, int64_t war, int64_t waw, double tau) {
   const double d_raw = n ? (double)raw / (double)n : 0.0;
   if (d_raw > tau) return JP_MODE_SEQ_RECOMMENDED;   // mode C
@@ -385,8 +396,15 @@ int32_t jp_select_mode(const jp_loop *L, const jp_profile *p, double tau_high) {
 // ---------------------------------------------------------------------------
 // static analysis lite (jp_static.cu)
 // ---------------------------------------------------------------------------
+// after_sample (nullable): called right after the prefix sample is launched,
+// before the host waits for it (jp_schedule queues side-stream work there)
 static jp_status static_check(const jp_loop *L, const Job &j, void *ws, const Layout &lo, jp_static *out,
-                              cudaStream_t st) {
+                              cudaStream_t st, const std::function<void()> *after_sample = nullptr) {
+  bool kicked = false;
+  auto kick = [&]() {
+    if (after_sample && !kicked) (*after_sample)();
+    kicked = true;
+  };
   memset(out, 0, sizeof *out);
   int64_t *hdr = at<int64_t>(ws, lo, R_HEADER);
   int *flags = reinterpret_cast<int *>(&hdr[H_AFFINE]);
@@ -395,11 +413,31 @@ static jp_status static_check(const jp_loop *L, const Job &j, void *ws, const La
     // there is not affine at all, and the full pass (a read of every index
     // array) is skipped -- the common case of indirect loops
     constexpr int kS = 64;
-    thread_local int32_t *pin = nullptr;
-    if (!pin && cudaMallocHost(&pin, 4 * kS * sizeof(int32_t)) != cudaSuccess) { pin = nullptr; cudaGetLastError(); }
-    const int32_t *qs[4] = {j.d.r, j.d.r2, j.d.w, j.d.s};
     const int m = (int)std::min<int64_t>(L->n, kS);
-    if (pin && m >= 3) {
+    TinyMirror &mm = tiny_mirror();
+    if (m >= 3 && mm.host) {
+      // verdict through mapped host words (tiny mirror [19], sequence [20]): one
+      // warp-sized kernel and a poll instead of copies and a stream sync
+      const unsigned long long seq = ++mm.seq;
+      JP_CUDA(launch_prefix_affine(j, m, reinterpret_cast<long long *>(mm.dev + 19), seq, st), "affine sample");
+      kick();
+      volatile unsigned long long *flag = reinterpret_cast<volatile unsigned long long *>(&mm.host[20]);
+      for (unsigned spins = 0; *flag != seq; spins++) {
+        if ((spins & 1023) == 1023) {
+          const cudaError_t q = cudaStreamQuery(st);
+          if (q != cudaSuccess && q != cudaErrorNotReady) return cuda_fail(q, "affine sample");
+          if (q == cudaSuccess && *flag != seq) return fail(JP_ERR_CUDA, "affine sample kernel did not publish");
+        }
+      }
+      if (*reinterpret_cast<volatile int64_t *>(&mm.host[19]) == 0) return JP_OK;   // out->affine == 0
+    }
+    thread_local int32_t *pin = nullptr;
+    if (!mm.host && !pin && cudaMallocHost(&pin, 4 * kS * sizeof(int32_t)) != cudaSuccess) {
+      pin = nullptr;
+      cudaGetLastError();
+    }
+    const int32_t *qs[4] = {j.d.r, j.d.r2, j.d.w, j.d.s};
+    if (!mm.host && pin && m >= 3) {
       for (int q = 0; q < 4; q++)
         if (qs[q]) JP_CUDA(cudaMemcpyAsync(pin + q * kS, qs[q], 4 * (size_t)m, cudaMemcpyDeviceToHost, st), "affine sample");
       JP_CUDA(cudaStreamSynchronize(st), "affine sample");
@@ -1779,12 +1817,35 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
     }
   };
   const bool pairs_ready = pdone != nullptr;
+  cudaEvent_t vdone = nullptr;
+  // every exit (an error return included) orders st after the side-stream clear
+  // of the shadow values and releases the event
+  struct JoinV {
+    cudaEvent_t &e; cudaStream_t s;
+    void join() { if (e) { cudaStreamWaitEvent(s, e, 0); cudaEventDestroy(e); e = nullptr; } }
+    ~JoinV() { join(); }
+  } join_v{vdone, st};
+  // the on-chip TLS shadow values must start at zero: cleared on a side stream
+  // queued right behind the static check's one-warp sample kernel (not before
+  // it: the clear would hold every SM while the host waits for the sample), so
+  // it overlaps the sample's round trip and the profile
+  const std::function<void()> clear_v = [&]() {
+    if (!(gfuse && (pairs || bucket)) || vdone) return;
+    auto *V = at<unsigned long long>(ws, lg, R_TLS_C_A);
+    if (V && cudaEventCreateWithFlags(&vdone, cudaEventDisableTiming) == cudaSuccess) {
+      cudaStream_t side = g_pool.get(40);
+      cudaEventRecord(vdone, st);          // after whatever ran before on st
+      cudaStreamWaitEvent(side, vdone, 0);
+      cudaMemsetAsync(V, 0, lg.bytes[R_TLS_C_A], side);
+      cudaEventRecord(vdone, side);
+    }
+  };
   if (c.static_check == 0 && ws) {
     // static analysis lite: affine, in-range, conflict-free -> DOALL without a profile
     Layout ls;
     if (jp_status e0 = check_ws(L, ws, ws_bytes, 0, ls)) { join_fill(); return e0; }
     jp_static sa;
-    if (jp_status e1 = static_check(L, j, ws, ls, &sa, st)) { join_fill(); return e1; }
+    if (jp_status e1 = static_check(L, j, ws, ls, &sa, st, &clear_v)) { join_fill(); return e1; }
     if (sa.independent && sa.in_range) {
       res->mode = JP_MODE_DOALL;
       res->profiled = 0;
@@ -1803,28 +1864,12 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
   int clean = 0;
   int64_t dist[32];
   bool have_dist = false;
-  cudaEvent_t vdone = nullptr;
-  // every exit (an error return included) orders st after the side-stream clear
-  // of the shadow values and releases the event
-  struct JoinV {
-    cudaEvent_t &e; cudaStream_t s;
-    void join() { if (e) { cudaStreamWaitEvent(s, e, 0); cudaEventDestroy(e); e = nullptr; } }
-    ~JoinV() { join(); }
-  } join_v{vdone, st};
+  bool spec = false;   // path 8 launched behind the profile, gated on its header
+  clear_v();   // (no static check ran)
+  if (vdone) clean = 2;
   if (gfuse) {
     // large A tables: stamped straight into {minW, minR} pairs (one 8-byte entry
     // per address for the classify lookups; the separate tables stay unwritten)
-    // the on-chip TLS shadow values must start at zero: clear them on a side
-    // stream while the (L2-atomic-bound) profile runs, instead of after it
-    auto *V = at<unsigned long long>(ws, lg, R_TLS_C_A);
-    if ((pairs || bucket) && V && cudaEventCreateWithFlags(&vdone, cudaEventDisableTiming) == cudaSuccess) {
-      cudaStream_t side = g_pool.get(40);
-      cudaEventRecord(vdone, st);          // after whatever ran before on st
-      cudaStreamWaitEvent(side, vdone, 0);
-      cudaMemsetAsync(V, 0, lg.bytes[R_TLS_C_A], side);
-      cudaEventRecord(vdone, side);
-      clean = 2;
-    }
     if (pairs) clean |= 1;   // region 7 holds this call's pair table, or the side stream's all-ones fill
     if (bucket) {
       // large A: the profile by address buckets (jp_bucket.cu), guide words included
@@ -1835,9 +1880,48 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
       else JP_TRY(jp_profile_stamp(L, ws, ws_bytes, stp));
       JP_CUDA(launch_prof_classify_guide(j, ws, lg, st, pairs), "profile classify");
     }
+    const bool vclear = vdone != nullptr;
     join_v.join();   // everything after the profile on st (TLS, or any later call) sees V zeroed
     int64_t h[H_DIST + 32];
-    JP_CUDA(d2h_small_sync(h, at<int64_t>(ws, lg, R_HEADER), sizeof h, st), "profile D2H");
+    int64_t *hd = at<int64_t>(ws, lg, R_HEADER);
+    // Path 8 launched behind the profile, before the host has read it: the
+    // kernel itself checks the header (gate) and runs only when Fig. 2(b) gives
+    // mode B with war = waw = 0 -- exactly when run_mode below would pick path 8
+    // -- so the GPU does not idle through the header's round trip; the header
+    // travels to the host on a side stream meanwhile.
+    spec = vclear && j.op == JP_OP_ADD_C && c.tls_path == 0 && c.tls_window == 0 && c.tls_recovery != 1 &&
+           L->n > 0 && !getenv("JP_TLS_NO_FLOW") && !getenv("JP_NO_SPEC_FLOW");
+    cudaEvent_t ep = nullptr, ec = nullptr;
+    if (spec && (cudaEventCreateWithFlags(&ep, cudaEventDisableTiming) != cudaSuccess ||
+                 cudaEventCreateWithFlags(&ec, cudaEventDisableTiming) != cudaSuccess)) {
+      if (ep) cudaEventDestroy(ep);
+      ep = nullptr;
+      spec = false;
+    }
+    if (spec) {
+      thread_local int64_t *pin = nullptr;
+      if (!pin && cudaMallocHost(reinterpret_cast<void **>(&pin), sizeof h) != cudaSuccess) pin = nullptr;
+      cudaError_t e = pin ? cudaSuccess : cudaErrorMemoryAllocation;
+      if (e == cudaSuccess) {
+        cudaStream_t side = g_pool.get(42);
+        cudaEventRecord(ep, st);
+        cudaStreamWaitEvent(side, ep, 0);
+        e = cudaMemcpyAsync(pin, hd, sizeof h, cudaMemcpyDeviceToHost, side);
+        if (e == cudaSuccess) e = cudaEventRecord(ec, side);
+      }
+      if (e == cudaSuccess) {
+        const uint32_t *g = at<uint32_t>(ws, lg, R_GUIDE);
+        e = launch_tls_flow(j, g, g + (L->n + 31) / 32, at<unsigned long long>(ws, lg, R_TLS_C_A),
+                            &hd[H_TLS_COMMITTED], st, nullptr, 0, hd, raw_max_for(L->n, c.tau_high));
+      }
+      if (e == cudaSuccess) e = cudaEventSynchronize(ec);
+      cudaEventDestroy(ep);
+      cudaEventDestroy(ec);
+      if (e != cudaSuccess) return cuda_fail(e, "profile D2H / one-window TLS");
+      memcpy(h, pin, sizeof h);
+    } else {
+      JP_CUDA(d2h_small_sync(h, hd, sizeof h, st), "profile D2H");
+    }
     if (h[H_BAD]) return fail(JP_ERR_INDEX, "%lld index entries are outside their arrays", (long long)h[H_BAD]);
     fill_profile(&p, L->n, h);
     memcpy(dist, h + H_DIST, sizeof dist);
@@ -1850,6 +1934,30 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
   res->mode = select_mode_counts(p.n, p.raw_iters, p.war_iters, p.waw_iters, c.tau_high);
   res->n_tasks = 1;
   res->n_batches = 1;
+  if (spec && res->mode == JP_MODE_TLS && p.war_iters == 0 && p.waw_iters == 0) {
+    // the gated path-8 kernel is running (its predicate is this one); its
+    // statistics are fixed by the profile: one window, the raw iterations are
+    // the violators (jp_tls_flow.cu).  JP_FLOW_CHECK=1 waits for it and checks
+    // that no violator lost its writer.
+    if (getenv("JP_FLOW_CHECK")) {
+      int64_t s4[4];
+      JP_CUDA(d2h_small_sync(s4, &at<int64_t>(ws, lg, R_HEADER)[H_TLS_COMMITTED], sizeof s4, st), "tls D2H");
+      if (s4[1] || s4[3] != p.raw_iters)
+        return fail(JP_ERR_ARG, "one-window TLS: %lld warps lost their writer, %lld violations for %lld raw iterations",
+                    (long long)s4[1], (long long)s4[3], (long long)p.raw_iters);
+    }
+    res->tls.committed = L->n;
+    res->tls.executed = L->n + p.raw_iters;
+    res->tls.windows = 1;
+    res->tls.violations = p.raw_iters;
+    res->tls_w_max = L->n;
+    res->tls_path = 8;
+    res->tls_guided = 1;
+    res->tls_recovery = JP_TLS_ONCHIP;
+    res->tls_cluster = num_sms();
+    res->task_mode_iters[JP_MODE_TLS] += L->n;
+    return JP_OK;
+  }
   return run_mode(L, j, res->mode, &p, c, ws, ws_bytes, res, st, gfuse && p.waw_iters == 0, clean,
                   have_dist ? dist : nullptr);
 }

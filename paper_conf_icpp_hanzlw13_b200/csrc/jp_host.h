@@ -70,8 +70,12 @@ bool bucket_profile_ok(const Job &j, void *ws, const Layout &lo);
 // wsrc (nullable) with lo: a range [lo, lo + n) of a loop whose profile recorded the
 // writer of every raw read (loop-local ids, wsrc indexed by the range's local i):
 // a raw read whose writer precedes the range reads A (committed) and is no violator
+// gate (nullable): a profile header the kernel checks before running (launched
+// ahead of the host's read of it): it exits at once unless H_BAD = H_WAR =
+// H_WAW = 0 and 0 < H_RAW <= raw_max
 cudaError_t launch_tls_flow(const Job &j, const uint32_t *graw, const uint32_t *gsrc, unsigned long long *V,
-                            int64_t *stats, cudaStream_t st, const int32_t *wsrc = nullptr, int64_t lo = 0);
+                            int64_t *stats, cudaStream_t st, const int32_t *wsrc = nullptr, int64_t lo = 0,
+                            const int64_t *gate = nullptr, int64_t raw_max = 0);
 // wsrc (nullable, ADD_C): the first writer of every raw iteration's read (int32 [n])
 // crange (nullable, needs chunk % 16384 == 0): per chunk the min and max address of A
 // the chunk touches (uint32 [2 * chunks]) -- the stealing scheduler's task ranges
@@ -147,6 +151,9 @@ cudaError_t launch_task_conflicts(const Job &j, const int32_t *chunk_task, int64
 
 // static analysis lite (jp_static.cu): flags[q] = index array q (r, r2, w, s) is affine
 cudaError_t launch_affine(const Job &j, int *flags, cudaStream_t st);
+// one warp: mir[0] = 1 when the first m (>= 2) entries of every index array are
+// affine, then mir[1] = seq (mapped host words, st.release.sys)
+cudaError_t launch_prefix_affine(const Job &j, int m, long long *mir, unsigned long long seq, cudaStream_t st);
 bool affine_conflict(int64_t af, int64_t bf, int64_t ag, int64_t bg, int64_t n);
 
 // tiny loops (jp_tiny.cu): the whole schedule in one CTA's shared memory

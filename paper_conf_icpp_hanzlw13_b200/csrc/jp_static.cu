@@ -62,6 +62,33 @@ cudaError_t launch_affine(const Job &j, int *flags, cudaStream_t st) {
   return launch_check();
 }
 
+// One warp: are the first m entries of every index array affine?  The verdict
+// goes to mapped host words (mir[0]), then the call's sequence number
+// (mir[1]): the host polls it instead of a device-to-host copy and a sync.
+__global__ void __launch_bounds__(32) k_prefix_affine(const int32_t *p0, const int32_t *p1, const int32_t *p2,
+                                                      const int32_t *p3, int m, long long *mir,
+                                                      unsigned long long seq) {
+  const int32_t *ps[4] = {p0, p1, p2, p3};
+  bool ok = true;
+#pragma unroll
+  for (int q = 0; q < 4; q++) {
+    if (!ps[q]) continue;
+    const int64_t b = __ldg(ps[q]), a = (int64_t)__ldg(ps[q] + 1) - b;
+    for (int k = threadIdx.x; k < m; k += 32) ok = ok && (int64_t)__ldg(ps[q] + k) == b + a * k;
+  }
+  ok = __all_sync(0xffffffffu, ok);
+  if (threadIdx.x == 0) {
+    mir[0] = ok ? 1 : 0;
+    asm volatile("st.release.sys.global.u64 [%0], %1;" ::"l"(mir + 1), "l"(seq) : "memory");
+  }
+}
+
+cudaError_t launch_prefix_affine(const Job &j, int m, long long *mir, unsigned long long seq, cudaStream_t st) {
+  k_prefix_affine<<<1, 32, 0, st>>>(j.d.r, j.d.r2, j.d.w, j.d.s, m, mir, seq);
+  note_launch();
+  return launch_check();
+}
+
 // ---------------------------------------------------------------------------
 // host: exact dependence test of two affine accesses f(i) = af*i + bf (a write)
 // and g(j) = ag*j + bg of the same array, i, j in [0, n), i != j

@@ -137,7 +137,12 @@ struct Flow {
 template <int DT>
 __global__ void __launch_bounds__(kFlowT, JP_FLOW_MINB) k_tls_flow(DLoop L, const uint32_t *graw, const uint32_t *gsrc,
                                                        unsigned long long *V, int64_t *stats, const int32_t *wsrc,
-                                                       uint32_t lo) {
+                                                       uint32_t lo, const int64_t *gate, int64_t raw_max) {
+  // gate (nullable): the profile header of this call -- launched before the host
+  // has read it, the kernel runs only if the profile makes the loop a path-8 loop
+  // (no bad index, war = waw = 0, 0 < raw <= raw_max, i.e. Fig. 2(b) mode B)
+  if (gate && (gate[H_BAD] != 0 || gate[H_WAR] != 0 || gate[H_WAW] != 0 || gate[H_RAW] <= 0 || gate[H_RAW] > raw_max))
+    return;
   Flow<DT> F;
   F.L = L; F.graw = graw; F.gsrc = gsrc; F.V = V; F.wsrc = wsrc; F.lo = lo;
   F.G = gridDim.x * (uint32_t)kFlowT;
@@ -168,7 +173,8 @@ __global__ void __launch_bounds__(kFlowT, JP_FLOW_MINB) k_tls_flow(DLoop L, cons
 
 template <int DT>
 static cudaError_t run_flow(const Job &j, const uint32_t *graw, const uint32_t *gsrc, unsigned long long *V,
-                            int64_t *stats, cudaStream_t st, const int32_t *wsrc, uint32_t lo) {
+                            int64_t *stats, cudaStream_t st, const int32_t *wsrc, uint32_t lo, const int64_t *gate,
+                            int64_t raw_max) {
   int maxb = 0;
   cudaOccupancyMaxActiveBlocksPerMultiprocessor(&maxb, (const void *)k_tls_flow<DT>, kFlowT, 0);
   if (maxb < 1) return cudaErrorInvalidConfiguration;
@@ -176,7 +182,7 @@ static cudaError_t run_flow(const Job &j, const uint32_t *graw, const uint32_t *
   const int64_t need = (j.d.n + kFlowT - 1) / kFlowT;
   if (need < grid) grid = (int)(need < 1 ? 1 : need);
   DLoop d = j.d;
-  void *args[] = {&d, &graw, &gsrc, &V, &stats, &wsrc, &lo};
+  void *args[] = {&d, &graw, &gsrc, &V, &stats, &wsrc, &lo, &gate, &raw_max};
   note_launch();
   return cudaLaunchCooperativeKernel((const void *)k_tls_flow<DT>, dim3(grid), dim3(kFlowT), args, 0, st);
 }
@@ -187,12 +193,13 @@ static cudaError_t run_flow(const Job &j, const uint32_t *graw, const uint32_t *
 // (committed n, executed n + violations, windows 1).  V must hold no value
 // tagged 1 << 32 for an address the loop writes (zeroed).
 cudaError_t launch_tls_flow(const Job &j, const uint32_t *graw, const uint32_t *gsrc, unsigned long long *V,
-                            int64_t *stats, cudaStream_t st, const int32_t *wsrc, int64_t lo) {
+                            int64_t *stats, cudaStream_t st, const int32_t *wsrc, int64_t lo, const int64_t *gate,
+                            int64_t raw_max) {
   cudaMemsetAsync(stats, 0, 4 * sizeof(int64_t), st);
   if (j.d.n == 0) return launch_check();
   if (j.op != JP_OP_ADD_C) return cudaErrorInvalidValue;
-  cudaError_t e = j.dt == JP_F32 ? run_flow<JP_F32>(j, graw, gsrc, V, stats, st, wsrc, (uint32_t)lo)
-                                 : run_flow<JP_I32>(j, graw, gsrc, V, stats, st, wsrc, (uint32_t)lo);
+  cudaError_t e = j.dt == JP_F32 ? run_flow<JP_F32>(j, graw, gsrc, V, stats, st, wsrc, (uint32_t)lo, gate, raw_max)
+                                 : run_flow<JP_I32>(j, graw, gsrc, V, stats, st, wsrc, (uint32_t)lo, gate, raw_max);
   if (e != cudaSuccess) return e;
   return launch_check();
 }

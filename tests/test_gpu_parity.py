@@ -1202,6 +1202,51 @@ def test_schedule_bucket_profile(case, buckets, monkeypatch):
     check_arrays(g, A, T)
 
 
+def _gate_cases():
+    n = (1 << 20) + 77
+    c3 = synth.config3(0.05, n=n)
+    raw = O.profile(to_oracle(c3))["raw_iters"]
+    cases = _bucket_cases()
+    return [("c3", c3, {}), ("doall", synth.config3(0.0, n=n), {}), ("rand_waw", cases[1][1], {}),
+            ("w_ident", cases[3][1], {}), ("seq", c3, {"tau_high": 0.01}),
+            ("tau_edge_tls", c3, {"tau_high": raw / n}), ("tau_edge_seq", c3, {"tau_high": (raw - 1) / n}),
+            ("forced_restart", c3, {"tls_recovery": 1})]
+
+
+@pytest.mark.parametrize("case", range(8))
+def test_schedule_gated_path8(case, monkeypatch):
+    """Path 8 launched behind the profile and gated on its header on the device
+    (jp_schedule, large A): the kernel runs exactly when Fig. 2(b) gives mode B
+    with war = waw = 0 -- the same result fields as the host-decided call
+    (JP_NO_SPEC_FLOW=1), arrays equal to the oracle, for loops on both sides of
+    the gate (DOALL, WAW, mode C, the tau_high edge, forced restart)."""
+    name, wl, kw = _gate_cases()[case]
+    _, A, T = O.run_seq(to_oracle(wl))
+    out = []
+    for spec in ("1", "0"):
+        if spec == "0":
+            monkeypatch.setenv("JP_NO_SPEC_FLOW", "1")
+        monkeypatch.setenv("JP_FLOW_CHECK", "1")
+        g = gpu(wl)
+        L = jp.Loop.from_workload(g)
+        ws = jp.workspace(L)
+        res = jp.jp_schedule(L, ws, **kw)
+        torch.cuda.synchronize()
+        check_arrays(g, A, T)
+        out.append(res)
+    a, b = out
+    assert a == b, (name, a, b)
+    if name in ("c3", "w_ident", "tau_edge_tls"):
+        assert a["mode_name"] == "TLS" and a["tls_path"] == 8, (name, a)
+        assert a["tls"]["violations"] == a["prof"]["raw_iters"] and a["tls"]["windows"] == 1
+    elif name in ("seq", "tau_edge_seq"):
+        assert a["mode"] == jp.JP_MODE_SEQ_RECOMMENDED and a["tls_path"] == 7, (name, a)
+    elif name == "doall":
+        assert a["mode"] == jp.JP_MODE_DOALL, a
+    else:
+        assert a["tls_path"] != 8, (name, a)
+
+
 def test_schedule_bucket_profile_bad_index():
     """An out-of-range index found by the bucket profile: JP_ERR_INDEX, nothing modified."""
     wl = synth.config3(0.01, n=(1 << 20) + 3)
