@@ -1299,7 +1299,12 @@ static jp_status task_conflicts(const Job &j, const jp_loop *L, void *ws, const 
   for (int t = 0; t < nt; t++)
     for (int64_t k = tasks[t].s / chunk; k * chunk < tasks[t].e; k++) ct[k] = t;
   int32_t *dct = reinterpret_cast<int32_t *>(sch + sl.chunk_task);
-  JP_CUDA(cudaMemcpyAsync(dct, ct.data(), 4 * nck, cudaMemcpyHostToDevice, st), "task map H2D");
+  bool dct_sent = false;
+  auto send_dct = [&]() -> cudaError_t {   // the chunk -> task map, for the device passes only
+    if (dct_sent) return cudaSuccess;
+    dct_sent = true;
+    return cudaMemcpyAsync(dct, ct.data(), 4 * nck, cudaMemcpyHostToDevice, st);
+  };
   // cheap sufficient test first: tasks with disjoint address ranges in every array never conflict
   if (!getenv("JP_TASK_MASKS_ALWAYS")) {
     std::vector<uint32_t> rg(4 * kMaxTasks);
@@ -1312,6 +1317,7 @@ static jp_status task_conflicts(const Job &j, const jp_loop *L, void *ws, const 
         }
     } else {
       uint32_t *drg = reinterpret_cast<uint32_t *>(sch + sl.ranges);
+      JP_CUDA(send_dct(), "task map H2D");
       JP_CUDA(launch_task_ranges(j, dct, chunk, drg, st), "task ranges");
       JP_CUDA(cudaMemcpyAsync(rg.data(), drg, 16 * kMaxTasks, cudaMemcpyDeviceToHost, st), "ranges D2H");
       JP_CUDA(cudaStreamSynchronize(st), "ranges sync");
@@ -1328,6 +1334,7 @@ static jp_status task_conflicts(const Job &j, const jp_loop *L, void *ws, const 
   }
   auto P = [&](size_t o) { return o == SIZE_MAX ? nullptr : reinterpret_cast<unsigned long long *>(sch + o); };
   unsigned long long *dconf = P(sl.conf);
+  JP_CUDA(send_dct(), "task map H2D");
   JP_CUDA(launch_task_conflicts(j, dct, chunk, nt, P(sl.wmA), P(sl.rmA), P(sl.wmT), P(sl.rmT), dconf, st),
           "conflicts");
   JP_CUDA(cudaMemcpyAsync(conf.data(), dconf, 8 * kMaxTasks, cudaMemcpyDeviceToHost, st), "conf D2H");
@@ -1361,12 +1368,28 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
   // (the write log of paths 5 / 6, unused by path 8)
   int32_t *wsrc = nullptr;
   uint32_t *crange = nullptr;   // per-chunk address ranges from the bucket profile (task PDG prefilter)
+  cudaEvent_t vev = nullptr;    // side-stream clear of the shadow values; every exit orders st after it
+  struct JoinVev {
+    cudaEvent_t &e; cudaStream_t s;
+    void join() { if (e) { cudaStreamWaitEvent(s, e, 0); cudaEventDestroy(e); e = nullptr; } }
+    ~JoinVev() { join(); }
+  } join_vev{vev, st};
   if (bucket_profile_ok(j, ws, lo)) {   // large A: the profile by address buckets (jp_bucket.cu)
     s_fresh = false;                    // (region 7 is not filled: the TLS task resets it)
     if (gbits && j.op == JP_OP_ADD_C && lo.bytes[R_TLS_S_A] >= 4 * (size_t)L->n && !getenv("JP_TLS_NO_FLOW"))
       wsrc = at<int32_t>(ws, lo, R_TLS_S_A);
     if (chunk % kBucketTile == 0 && !getenv("JP_TASK_MASKS_ALWAYS"))
       crange = reinterpret_cast<uint32_t *>(sch + sl.crange);
+    // the shadow values of a one-window TLS task start at zero: cleared on a
+    // side stream while the profile runs
+    auto *V = at<unsigned long long>(ws, lo, R_TLS_C_A);
+    if (wsrc && V && cudaEventCreateWithFlags(&vev, cudaEventDisableTiming) == cudaSuccess) {
+      cudaStream_t side = g_pool.get(40);
+      cudaEventRecord(vev, st);
+      cudaStreamWaitEvent(side, vev, 0);
+      cudaMemsetAsync(V, 0, lo.bytes[R_TLS_C_A], side);
+      cudaEventRecord(vev, side);
+    }
     JP_CUDA(launch_prof_bucket(j, ws, lo, gbits, gbits ? gbits + (L->n + 31) / 32 : nullptr, chunk, cc, st, wsrc,
                                crange),
             "profile (buckets)");
@@ -1377,13 +1400,33 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
   }
   std::vector<int64_t> hc(3 * nck), h(8);
   std::vector<uint32_t> hcr;
-  JP_CUDA(cudaMemcpyAsync(hc.data(), cc, 24 * nck, cudaMemcpyDeviceToHost, st), "chunk D2H");
-  if (crange) {
-    hcr.resize(2 * nck);
-    JP_CUDA(cudaMemcpyAsync(hcr.data(), crange, 8 * nck, cudaMemcpyDeviceToHost, st), "chunk ranges D2H");
+  {
+    // chunk counts, chunk address ranges and the header through one pinned
+    // staging buffer (pageable copies each stall the host)
+    thread_local char *pin = nullptr;
+    thread_local size_t pin_bytes = 0;
+    const size_t need = 24 * (size_t)nck + (crange ? 8 * (size_t)nck : 0) + 64;
+    if (need > pin_bytes) {
+      if (pin) cudaFreeHost(pin);
+      pin = nullptr;
+      pin_bytes = 0;
+      if (cudaMallocHost(reinterpret_cast<void **>(&pin), need) == cudaSuccess) pin_bytes = need;
+      else cudaGetLastError();
+    }
+    char *dst_c = pin ? pin : reinterpret_cast<char *>(hc.data());
+    if (crange) hcr.resize(2 * nck);
+    char *dst_r = pin ? pin + 24 * nck : reinterpret_cast<char *>(hcr.data());
+    char *dst_h = pin ? pin + 24 * nck + (crange ? 8 * nck : 0) : reinterpret_cast<char *>(h.data());
+    JP_CUDA(cudaMemcpyAsync(dst_c, cc, 24 * nck, cudaMemcpyDeviceToHost, st), "chunk D2H");
+    if (crange) JP_CUDA(cudaMemcpyAsync(dst_r, crange, 8 * nck, cudaMemcpyDeviceToHost, st), "chunk ranges D2H");
+    JP_CUDA(cudaMemcpyAsync(dst_h, at<int64_t>(ws, lo, R_HEADER), 64, cudaMemcpyDeviceToHost, st), "profile D2H");
+    JP_CUDA(cudaStreamSynchronize(st), "profile sync");
+    if (pin) {
+      memcpy(hc.data(), dst_c, 24 * nck);
+      if (crange) memcpy(hcr.data(), dst_r, 8 * nck);
+      memcpy(h.data(), dst_h, 64);
+    }
   }
-  JP_CUDA(cudaMemcpyAsync(h.data(), at<int64_t>(ws, lo, R_HEADER), 64, cudaMemcpyDeviceToHost, st), "profile D2H");
-  JP_CUDA(cudaStreamSynchronize(st), "profile sync");
   if (h[H_BAD]) return fail(JP_ERR_INDEX, "%lld index entries are outside their arrays", (long long)h[H_BAD]);
   fill_profile(&res->prof, L->n, h.data());
   res->profiled = 1;
@@ -1413,14 +1456,20 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
   const bool guided_ok = gfuse;
   std::vector<int> grid_tls;   // on-chip TLS tasks, run on every SM after the batch's other tasks
   std::vector<int> flow_tasks;  // ... of them, run as one window (path 8): stats completed on the host
-  bool v_zeroed = false;
+  // the side-stream clear (done long before: it overlapped the profile) is
+  // joined before any task runs
+  const bool v_zeroed_side = vev != nullptr;
+  join_vev.join();
+  bool v_zeroed = v_zeroed_side;
   cudaEvent_t ev0;
   JP_CUDA(cudaEventCreateWithFlags(&ev0, cudaEventDisableTiming), "event");
   std::vector<cudaEvent_t> evs;
   std::vector<int> tls_tasks;
   for (int lv = 0; lv < nlev; lv++) {
     bool any_priv = false;
-    for (int t = 0; t < nt; t++) any_priv |= level[t] == lv && tasks[t].mode == JP_MODE_PRIVATIZED;
+    int n_priv = 0;
+    for (int t = 0; t < nt; t++) n_priv += level[t] == lv && tasks[t].mode == JP_MODE_PRIVATIZED;
+    any_priv = n_priv > 0;
     // the element ranges this batch's privatized tasks can write (their keys):
     // the whole arrays unless the range prefilter ran
     int64_t kA0 = 0, kA1 = L->len_A, kT0 = 0, kT1 = L->len_T;
@@ -1441,10 +1490,13 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
     }
     auto *keysA = at<unsigned long long>(ws, lo, R_KEYS_A);
     auto *keysT = at<unsigned long long>(ws, lo, R_KEYS_T);
-    if (any_priv) {
-      if (keysA && kA1 > kA0) cudaMemsetAsync(keysA + kA0, 0, 8 * (size_t)(kA1 - kA0), st);
-      if (keysT && kT1 > kT0) cudaMemsetAsync(keysT + kT0, 0, 8 * (size_t)(kT1 - kT0), st);
-    }
+    // the key ranges start at zero: cleared on the privatized task's own stream
+    // when the batch has one (the other tasks start at once), else before the batch
+    auto clear_keys = [&](cudaStream_t s) {
+      if (keysA && kA1 > kA0) cudaMemsetAsync(keysA + kA0, 0, 8 * (size_t)(kA1 - kA0), s);
+      if (keysT && kT1 > kT0) cudaMemsetAsync(keysT + kT0, 0, 8 * (size_t)(kT1 - kT0), s);
+    };
+    if (n_priv > 1) clear_keys(st);
     cudaEventRecord(ev0, st);
     int sidx = 0;
     std::vector<cudaEvent_t> joins;
@@ -1487,6 +1539,7 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
           }
           tls_tasks.push_back(t);
         } else if (tasks[t].mode == JP_MODE_PRIVATIZED) {
+          if (n_priv == 1) clear_keys(s2);
           JP_CUDA(launch_priv_stream(sj, ws, lo, false, s2), "priv task");
         } else {
           JP_CUDA(launch_doall(sj, s2), "doall task");
@@ -1543,6 +1596,7 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
                                     tstats + 4 * t, st, s_fresh ? 1 : 0),
                 "tls task");
         s_fresh = false;
+        v_zeroed = false;   // path 6 leaves its shadow values in V
       } else {
         JP_CUDA(launch_tls_fwd(sj, tp.window, tp.cluster, b0, b1, tstats + 4 * t, st), "tls task");
       }
@@ -1912,7 +1966,8 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
       if (e == cudaSuccess) {
         const uint32_t *g = at<uint32_t>(ws, lg, R_GUIDE);
         e = launch_tls_flow(j, g, g + (L->n + 31) / 32, at<unsigned long long>(ws, lg, R_TLS_C_A),
-                            &hd[H_TLS_COMMITTED], st, nullptr, 0, hd, raw_max_for(L->n, c.tau_high));
+                            &hd[H_TLS_COMMITTED], st, nullptr, 0, hd, raw_max_for(L->n, c.tau_high),
+                            !bucket);   // (the bucket profile's reset of the header zeroed the statistics)
       }
       if (e == cudaSuccess) e = cudaEventSynchronize(ec);
       cudaEventDestroy(ep);

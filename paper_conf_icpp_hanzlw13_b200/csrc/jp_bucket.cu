@@ -34,6 +34,7 @@
 // per iteration (raw from the read, war / waw from the write); SAXPY's only A
 // access is Y[w], read and written by the same iteration, so raw = war = waw =
 // "an earlier iteration wrote this address" (one write record).
+#include <algorithm>
 #include "jp_host.h"
 
 namespace jp {
@@ -404,9 +405,25 @@ __global__ void __launch_bounds__(kEvalThreads) k_bk_eval(BkView V, const uint32
       if (s_cc[k]) atomicAdd(reinterpret_cast<unsigned long long *>(&O.cc[k]), (unsigned long long)s_cc[k]);
 }
 
-__global__ void k_bk_init_ranges(uint32_t *cr, int64_t nck) {
-  const int64_t c = (int64_t)blockIdx.x * blockDim.x + threadIdx.x;
-  if (c < nck) { cr[2 * c] = 0xFFFFFFFFu; cr[2 * c + 1] = 0u; }
+// everything the profile accumulates into, reset in one launch: the header
+// (first raw iteration = -1), the guide words, the per-chunk counts and the
+// per-chunk address ranges (min = ~0, max = 0)
+__global__ void __launch_bounds__(256) k_bk_prep(int64_t *hdr, uint32_t *graw, uint32_t *gsrc, int64_t nw, int64_t *cc,
+                                                 int64_t ncc, uint32_t *cr, int64_t nck) {
+  const int64_t nh = (int64_t)(kHeaderBytes / 8);
+  int64_t m = nh;
+  if (nw > m) m = nw;
+  if (ncc > m) m = ncc;
+  if (nck > m) m = nck;
+  for (int64_t k = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; k < m; k += (int64_t)gridDim.x * blockDim.x) {
+    if (k < nh) hdr[k] = k == H_FIRST_RAW ? -1 : 0;
+    if (k < nw) {
+      if (graw) graw[k] = 0;
+      if (gsrc) gsrc[k] = 0;
+    }
+    if (cc && k < ncc) cc[k] = 0;
+    if (cr && k < nck) { cr[2 * k] = 0xFFFFFFFFu; cr[2 * k + 1] = 0u; }
+  }
 }
 
 namespace {
@@ -482,20 +499,22 @@ cudaError_t launch_prof_bucket(const Job &j, void *ws, const Layout &lo, uint32_
   BkPlan P;
   if (!plan(j, ws, lo, P)) return cudaErrorInvalidValue;
   static_assert(kTile == kBucketTile, "jp_host.h kBucketTile");
+  int64_t nck = 0;
   if (crange && chunk > 0 && chunk % kTile == 0) {
-    const int64_t nck = (j.d.n + chunk - 1) / chunk;
-    k_bk_init_ranges<<<(int)((nck + 255) / 256), 256, 0, st>>>(crange, nck);   // min = ~0, max = 0
-    note_launch();
+    nck = (j.d.n + chunk - 1) / chunk;
     P.v.crange = crange;
     P.v.ctiles = (int)(chunk / kTile);
   }
   int64_t *hdr = at<int64_t>(ws, lo, R_HEADER);
-  cudaMemsetAsync(hdr, 0, kHeaderBytes, st);
-  cudaMemsetAsync(&hdr[H_FIRST_RAW], 0xFF, sizeof(int64_t), st);
   const int64_t nw = (j.d.n + 31) / 32;
-  if (graw) cudaMemsetAsync(graw, 0, 4 * (size_t)nw, st);
-  if (gsrc) cudaMemsetAsync(gsrc, 0, 4 * (size_t)nw, st);
-  if (cc) cudaMemsetAsync(cc, 0, sizeof(int64_t) * 3 * ((j.d.n + chunk - 1) / chunk), st);
+  const int64_t ncc = cc ? 3 * ((j.d.n + chunk - 1) / chunk) : 0;
+  {
+    int64_t m = std::max<int64_t>(std::max<int64_t>((int64_t)(kHeaderBytes / 8), nw), std::max(ncc, nck));
+    const int64_t need = (m + 255) / 256, cap = (int64_t)num_sms() * 4;
+    k_bk_prep<<<(int)(need < cap ? need : cap), 256, 0, st>>>(hdr, graw, gsrc, nw, cc, ncc, nck ? crange : nullptr,
+                                                              nck);
+    note_launch();
+  }
   BkOut O{hdr, graw, gsrc, chunk, cc, j.d.base, j.op == JP_OP_ADD_C ? wsrc : nullptr};
   if (j.op == JP_OP_ADD_C) run_bucket<JP_OP_ADD_C>(P, j.d, hdr, O, st);
   else run_bucket<JP_OP_SAXPY>(P, j.d, hdr, O, st);

@@ -75,7 +75,7 @@ bool bucket_profile_ok(const Job &j, void *ws, const Layout &lo);
 // H_WAW = 0 and 0 < H_RAW <= raw_max
 cudaError_t launch_tls_flow(const Job &j, const uint32_t *graw, const uint32_t *gsrc, unsigned long long *V,
                             int64_t *stats, cudaStream_t st, const int32_t *wsrc = nullptr, int64_t lo = 0,
-                            const int64_t *gate = nullptr, int64_t raw_max = 0);
+                            const int64_t *gate = nullptr, int64_t raw_max = 0, bool zero_stats = true);
 // wsrc (nullable, ADD_C): the first writer of every raw iteration's read (int32 [n])
 // crange (nullable, needs chunk % 16384 == 0): per chunk the min and max address of A
 // the chunk touches (uint32 [2 * chunks]) -- the stealing scheduler's task ranges

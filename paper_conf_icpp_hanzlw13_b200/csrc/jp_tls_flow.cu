@@ -194,8 +194,8 @@ static cudaError_t run_flow(const Job &j, const uint32_t *graw, const uint32_t *
 // tagged 1 << 32 for an address the loop writes (zeroed).
 cudaError_t launch_tls_flow(const Job &j, const uint32_t *graw, const uint32_t *gsrc, unsigned long long *V,
                             int64_t *stats, cudaStream_t st, const int32_t *wsrc, int64_t lo, const int64_t *gate,
-                            int64_t raw_max) {
-  cudaMemsetAsync(stats, 0, 4 * sizeof(int64_t), st);
+                            int64_t raw_max, bool zero_stats) {
+  if (zero_stats) cudaMemsetAsync(stats, 0, 4 * sizeof(int64_t), st);
   if (j.d.n == 0) return launch_check();
   if (j.op != JP_OP_ADD_C) return cudaErrorInvalidValue;
   cudaError_t e = j.dt == JP_F32 ? run_flow<JP_F32>(j, graw, gsrc, V, stats, st, wsrc, (uint32_t)lo, gate, raw_max)
