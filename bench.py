@@ -347,7 +347,7 @@ def modes_sweep(jp, dev, st):
     #  restart_*: the same with restart recovery (reading A6: prefix commit, restart at the first violator)
     tls = []
     names = {1: "cta", 2: "grid", 3: "cluster16", 4: "tiny", 5: "onchip-cluster", 6: "onchip-grid",
-             7: "serial-warp", 8: "onchip-one-window"}
+             7: "serial-warp", 8: "onchip-one-window", 9: "onchip-one-window-waw"}
 
     def timed(fn, A, A0, reps=None):
         """warm up, then the median of `reps` timed runs (20, or
@@ -405,8 +405,10 @@ def modes_sweep(jp, dev, st):
         del wl, ws, L, A0
     out["config3_tls_delta_2e20"] = sens
     # config 3's shape WITH write-after-write (synth.config3_waw: w 2-to-1 onto half
-    # the addresses): on-chip recovery (reading B7) is illegal, so jp_schedule runs
-    # restart TLS (reading A6) with the cap / path of the distance-hazard plan
+    # the addresses): jp_schedule runs the one-window on-chip TLS fed by the last
+    # earlier writer of every raw read (path 9, reading B14); the restart form
+    # (reading A6, tls_recovery = 1, cap / path from the distance-hazard plan)
+    # beside it
     waw = []
     for delta in (1024, 1 << 20):
         for d in (0.001, 0.01, 0.05, 0.10):
@@ -414,15 +416,20 @@ def modes_sweep(jp, dev, st):
             A0 = wl.A.clone()
             L = jp.Loop.from_workload(wl)
             ws = jp.workspace(L)
-            res, ms = timed(lambda: jp.jp_schedule(L, ws, stream=st), wl.A, A0)
-            waw.append({"density": d, "delta": delta, "mode": res["mode_name"], "ms": ms,
-                        "committed_per_s": wl.n / (ms * 1e-3), "raw_iters": res["prof"]["raw_iters"],
-                        "waw_iters": res["prof"]["waw_iters"], "windows": res["tls"]["windows"],
-                        "violations": res["tls"]["violations"], "recovery": ["restart", "onchip"][res["tls_recovery"]],
-                        "tls_w_max": res["tls_w_max"], "tls_path": names.get(res["tls_path"], "?"),
-                        "us_per_window": ms * 1e3 / max(res["tls"]["windows"], 1)})
+            row = {"density": d, "delta": delta}
+            for tag, rec in (("", 0), ("restart_", 1)):
+                res, ms = timed(lambda: jp.jp_schedule(L, ws, stream=st, tls_recovery=rec), wl.A, A0)
+                row["raw_iters"] = res["prof"]["raw_iters"]
+                row["waw_iters"] = res["prof"]["waw_iters"]
+                row[tag + "schedule"] = {
+                    "mode": res["mode_name"], "ms": ms, "committed_per_s": wl.n / (ms * 1e-3),
+                    "windows": res["tls"]["windows"], "violations": res["tls"]["violations"],
+                    "recovery": ["restart", "onchip"][res["tls_recovery"]], "tls_w_max": res["tls_w_max"],
+                    "tls_path": names.get(res["tls_path"], "?"),
+                    "us_per_window": ms * 1e3 / max(res["tls"]["windows"], 1)}
+            waw.append(row)
             del wl, ws, L, A0
-    out["config3_waw_restart"] = waw
+    out["config3_waw"] = waw
     out["crossover"] = crossover_sweep(jp, dev, st)
     # config 4: privatized.  The whole jp_schedule call (what a user runs: reading
     # B11 decides privatized without a profile, the s indices are checked on the

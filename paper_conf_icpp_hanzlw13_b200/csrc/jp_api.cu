@@ -2013,6 +2013,42 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
     res->task_mode_iters[JP_MODE_TLS] += L->n;
     return JP_OK;
   }
+  // an ADD_C TLS loop WITH WAR / WAW, profiled by address buckets: the last
+  // earlier writer of every raw read from the records still in place, then one
+  // window over the whole loop (path 9, reading B14, jp_tls_flow.cu); the
+  // windowed paths stay for what the last-writer pass cannot hold
+  if (bucket && res->mode == JP_MODE_TLS && j.op == JP_OP_ADD_C && (p.war_iters > 0 || p.waw_iters > 0) &&
+      c.tls_recovery == 0 && c.tls_path == 0 && c.tls_window == 0 && !getenv("JP_TLS_NO_FLOW")) {
+    int64_t *hd = at<int64_t>(ws, lg, R_HEADER);
+    auto *pred = at<int32_t>(ws, lg, R_TLS_S_A);
+    auto *bits = reinterpret_cast<uint32_t *>(pred + ((L->n + 63) & ~(int64_t)63));
+    auto *V = at<unsigned long long>(ws, lg, R_TLS_C_A);
+    const uint32_t *graw = at<uint32_t>(ws, lg, R_GUIDE);
+    if (!(clean & 2)) JP_CUDA(cudaMemsetAsync(V, 0, 8 * (size_t)L->n, st), "shadow clear");
+    JP_CUDA(launch_prof_pred(j, ws, lg, pred, bits, st), "last writers");
+    JP_CUDA(launch_tls_flow_waw(j, graw, pred, bits, V, &hd[H_TLS_COMMITTED], hd, st), "tls one window (waw)");
+    int64_t h2[H_PRED_SEG + 1];
+    JP_CUDA(d2h_small_sync(h2, hd, sizeof h2, st), "tls D2H");
+    if (h2[H_PRED_FAIL] == 0) {
+      if (h2[H_TLS_EXECUTED])
+        return fail(JP_ERR_ARG, "one-window TLS: a violator's writer never published (profile inconsistent)");
+      if (h2[H_TLS_VIOL] != p.raw_iters)
+        return fail(JP_ERR_ARG, "one-window TLS: %lld violations for %lld raw iterations",
+                    (long long)h2[H_TLS_VIOL], (long long)p.raw_iters);
+      res->tls.committed = L->n;
+      res->tls.executed = L->n + p.raw_iters;
+      res->tls.windows = 1;
+      res->tls.violations = p.raw_iters;
+      res->tls_w_max = L->n;
+      res->tls_path = 9;
+      res->tls_guided = 1;
+      res->tls_recovery = JP_TLS_ONCHIP;
+      res->tls_cluster = num_sms();
+      res->task_mode_iters[JP_MODE_TLS] += L->n;
+      return JP_OK;
+    }
+    clean &= ~1;   // region 7 now holds the pass's tables; V is untouched (the kernel exited)
+  }
   return run_mode(L, j, res->mode, &p, c, ws, ws_bytes, res, st, gfuse && p.waw_iters == 0, clean,
                   have_dist ? dist : nullptr);
 }

@@ -405,6 +405,152 @@ __global__ void __launch_bounds__(kEvalThreads) k_bk_eval(BkView V, const uint32
       if (s_cc[k]) atomicAdd(reinterpret_cast<unsigned long long *>(&O.cc[k]), (unsigned long long)s_cc[k]);
 }
 
+// ---------------------------------------------------------------------------
+// The last earlier writer of every raw read (reading B14, path 9).  With WAW a
+// raw read of address a at iteration i must see the value of
+// pred(i) = max{ j < i : w[j] = a } (the sequential semantics);
+// the first-writer tables above do not hold it.  One CTA per bucket, over the
+// records the profile left in place:
+//   count    writers per address (shared atomics);
+//   scan     the address segments of a writer list;
+//   fill     every writer's iteration into its address's segment (unordered);
+//   reads    pred(i) = the largest listed writer below i -> pred[i], and the
+//            writer's publish bit; a read with no earlier writer of an address
+//            that IS written (an exposed read, WAR on the window-start value)
+//            marks the address;
+//   writers  per address, its last writer: commit at once (now) or, when the
+//            address has an exposed read, after the flow kernel's barrier (later).
+// A bucket whose writers do not fit shared memory, or an address with more than
+// kPredSegCap writers, fails the pass (H_PRED_FAIL): the caller keeps the
+// windowed paths.  ADD_C only (one exposed read, one write per iteration).
+// ---------------------------------------------------------------------------
+// Two tiers: 512-thread CTAs, two per SM, hold up to kPredCapS writers per bucket;
+// a bucket with more is marked and redone by the second launch (1024 threads,
+// one CTA per SM, the whole 226 KB), which skips every other bucket.
+constexpr uint32_t kPredSegCap = 4096;
+constexpr size_t kPredSmemS = 110 * 1024, kPredSmemB = 226 * 1024;   // (+ static <= the 227 KB opt-in)
+constexpr size_t kPredFixed = 4 * (size_t)kBSpan + kBSpan / 8;      // segment ends + exposed-read flags
+constexpr uint32_t kPredCapS = (uint32_t)((kPredSmemS - kPredFixed) / 4);
+constexpr uint32_t kPredCapB = (uint32_t)((kPredSmemB - kPredFixed) / 4);
+
+struct PredOut {
+  int32_t *pred;                  // [n] last earlier writer of raw iteration i's read (loop-local)
+  uint32_t *pub, *now, *later;    // [nw] each, zeroed by the caller
+  int64_t *hdr;                   // H_PRED_FAIL, H_PRED_SEG
+  uint32_t *redo;                 // [B] bucket left to the big tier
+};
+
+template <bool BIG>
+__global__ void __launch_bounds__(BIG ? 1024 : 512, BIG ? 1 : 2) k_bk_pred(BkView V, const uint32_t *base,
+                                                                           const uint32_t *tot,
+                                                                           const unsigned long long *rec, PredOut O) {
+  constexpr int kT = BIG ? 1024 : 512;
+  constexpr uint32_t kCap = BIG ? kPredCapB : kPredCapS;
+  extern __shared__ uint32_t s_dyn[];
+  // cur[a]: first the writer count of address a, then (scan) the start of its
+  // segment, then (fill) its end -- segment a is [cur[a-1], cur[a])
+  uint32_t *cur = s_dyn;                    // [kBSpan]
+  uint32_t *xflag = cur + kBSpan;           // [kBSpan / 32] address has an exposed read
+  uint32_t *wl = xflag + kBSpan / 32;       // [kCap] writer lists
+  __shared__ uint32_t s_wsum[kT / 32];
+  __shared__ uint32_t s_nw;
+  const int b = blockIdx.x;
+  if (BIG && !O.redo[b]) return;
+  const uint32_t total = tot[b];
+  const unsigned long long *rb = rec + base[b];
+  for (int k = threadIdx.x; k < kBSpan; k += kT) cur[k] = 0;
+  for (int k = threadIdx.x; k < kBSpan / 32; k += kT) xflag[k] = 0;
+  __syncthreads();
+  constexpr int kU = 4;
+  auto sweep = [&](auto &&f) {
+    for (uint32_t p0 = threadIdx.x; p0 < total; p0 += kT * kU) {
+      unsigned long long xv[kU];
+#pragma unroll
+      for (int u = 0; u < kU; u++) {
+        const uint32_t p = p0 + (uint32_t)u * kT;
+        xv[u] = p < total ? rb[p] : 0ull;
+      }
+#pragma unroll
+      for (int u = 0; u < kU; u++)
+        if (p0 + (uint32_t)u * kT < total) f(xv[u]);
+    }
+  };
+  sweep([&](unsigned long long x) {
+    if (x & kRecW) atomicAdd(&cur[(uint32_t)(x >> 32) & (kBSpan - 1)], 1u);
+  });
+  __syncthreads();
+  // exclusive scan of the counts: kPer addresses per thread
+  constexpr int kPer = kBSpan / kT;
+  const int a0 = threadIdx.x * kPer;
+  uint32_t c[kPer], s = 0, mseg = 0;
+#pragma unroll
+  for (int k = 0; k < kPer; k++) {
+    c[k] = cur[a0 + k];
+    s += c[k];
+    mseg = max(mseg, c[k]);
+  }
+  uint32_t x = s;
+  for (int o = 1; o < 32; o <<= 1) {
+    const uint32_t y = __shfl_up_sync(0xffffffffu, x, o);
+    if ((threadIdx.x & 31) >= o) x += y;
+  }
+  if ((threadIdx.x & 31) == 31) s_wsum[threadIdx.x >> 5] = x;
+  mseg = __reduce_max_sync(0xffffffffu, mseg);
+  __syncthreads();
+  uint32_t run = x - s;
+  for (int k = 0; k < (int)(threadIdx.x >> 5); k++) run += s_wsum[k];
+#pragma unroll
+  for (int k = 0; k < kPer; k++) {
+    cur[a0 + k] = run;
+    run += c[k];
+  }
+  if (threadIdx.x == kT - 1) s_nw = run;
+  if ((threadIdx.x & 31) == 0 && mseg)
+    atomicMax(reinterpret_cast<unsigned long long *>(&O.hdr[H_PRED_SEG]), (unsigned long long)mseg);
+  __syncthreads();
+  const uint32_t nwr = s_nw;
+  if (nwr == 0) return;   // nothing written in this bucket: no read has a writer
+  if (nwr > kCap || __syncthreads_or(mseg > kPredSegCap)) {
+    if (threadIdx.x == 0) {
+      if (!BIG && nwr > kCap && mseg <= kPredSegCap) O.redo[b] = 1;
+      else atomicAdd(reinterpret_cast<unsigned long long *>(&O.hdr[H_PRED_FAIL]), 1ull);
+    }
+    return;
+  }
+  sweep([&](unsigned long long x) {
+    if (x & kRecW) wl[atomicAdd(&cur[(uint32_t)(x >> 32) & (kBSpan - 1)], 1u)] = (uint32_t)x;
+  });
+  __syncthreads();
+  // reads: the largest writer below i in the address's list
+  sweep([&](unsigned long long x) {
+    if (x & kRecW) return;
+    const uint32_t i = (uint32_t)x, al = (uint32_t)(x >> 32) & (kBSpan - 1);
+    const uint32_t p0 = al ? cur[al - 1] : 0u, p1 = cur[al];
+    if (p0 == p1) return;   // an address nobody writes
+    uint32_t best = 0xFFFFFFFFu;
+    for (uint32_t p = p0; p < p1; p++) {
+      const uint32_t j = wl[p];
+      if (j < i && (best == 0xFFFFFFFFu || j > best)) best = j;
+    }
+    if (best != 0xFFFFFFFFu) {
+      O.pred[i] = (int32_t)best;
+      atomicOr(&O.pub[best >> 5], 1u << (best & 31));
+    } else {
+      atomicOr(&xflag[al >> 5], 1u << (al & 31));
+    }
+  });
+  __syncthreads();
+  // writers: the last writer of every written address commits
+  for (int al = threadIdx.x; al < kBSpan; al += kT) {
+    const uint32_t p0 = al ? cur[al - 1] : 0u, p1 = cur[al];
+    if (p0 == p1) continue;
+    uint32_t last = wl[p0];
+    for (uint32_t p = p0 + 1; p < p1; p++) last = max(last, wl[p]);
+    uint32_t *bits = (xflag[al >> 5] >> (al & 31)) & 1u ? O.later : O.now;
+    atomicOr(&bits[last >> 5], 1u << (last & 31));
+  }
+}
+
 // everything the profile accumulates into, reset in one launch: the header
 // (first raw iteration = -1), the guide words, the per-chunk counts and the
 // per-chunk address ranges (min = ~0, max = 0)
@@ -453,13 +599,9 @@ bool plan(const Job &j, void *ws, const Layout &lo, BkPlan &P) {
   // profile keeps no tables, and every privatized run clears the keys it
   // applies); offsets in maxRx_A (free until a jp_tls_guide pass, which
   // jp_schedule skips)
-  size_t rb = 0, endo = lo.off[R_MINW_A];
-  for (int r = R_MINW_A; r <= R_KEYS_A; r++) {
-    if (!lo.bytes[r]) continue;
-    if (lo.off[r] != endo) break;
-    rb += lo.bytes[r];
-    endo = lo.off[r] + lo.bytes[r];
-  }
+  // (the regions follow one another in layout order, separated only by the
+  // 256-byte alignment padding of the workspace: the span is one free piece)
+  const size_t rb = lo.bytes[R_KEYS_A] ? lo.off[R_KEYS_A] + lo.bytes[R_KEYS_A] - lo.off[R_MINW_A] : 0;
   if (!lo.bytes[R_MINW_A] || rb < 8 * (size_t)nrec) return false;
   if (lo.bytes[R_MAXRX_A] < 4 * ((size_t)T * B + 2 * (size_t)B)) return false;
   P.v = BkView{d.r, d.w, d.n, d.ioff, (uint32_t)d.lenA, B, T, nullptr, 1};
@@ -518,6 +660,26 @@ cudaError_t launch_prof_bucket(const Job &j, void *ws, const Layout &lo, uint32_
   BkOut O{hdr, graw, gsrc, chunk, cc, j.d.base, j.op == JP_OP_ADD_C ? wsrc : nullptr};
   if (j.op == JP_OP_ADD_C) run_bucket<JP_OP_ADD_C>(P, j.d, hdr, O, st);
   else run_bucket<JP_OP_SAXPY>(P, j.d, hdr, O, st);
+  return launch_check();
+}
+
+cudaError_t launch_prof_pred(const Job &j, void *ws, const Layout &lo, int32_t *pred, uint32_t *bits,
+                             cudaStream_t st) {
+  BkPlan P;
+  if (j.op != JP_OP_ADD_C || !plan(j, ws, lo, P)) return cudaErrorInvalidValue;
+  const int64_t nw = (j.d.n + 31) / 32;
+  cudaError_t e = cudaMemsetAsync(bits, 0, 3 * 4 * (size_t)nw, st);
+  // redo flags in the per-tile offsets (P.cnt: the scatter was their last reader)
+  if (e == cudaSuccess) e = cudaMemsetAsync(P.cnt, 0, 4 * (size_t)P.v.B, st);
+  if (e == cudaSuccess)
+    e = cudaFuncSetAttribute(k_bk_pred<false>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)kPredSmemS);
+  if (e == cudaSuccess)
+    e = cudaFuncSetAttribute(k_bk_pred<true>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)kPredSmemB);
+  if (e != cudaSuccess) return e;
+  PredOut O{pred, bits, bits + nw, bits + 2 * nw, at<int64_t>(ws, lo, R_HEADER), P.cnt};
+  k_bk_pred<false><<<P.v.B, 512, kPredSmemS, st>>>(P.v, P.base, P.tot, P.rec, O);
+  k_bk_pred<true><<<P.v.B, 1024, kPredSmemB, st>>>(P.v, P.base, P.tot, P.rec, O);
+  note_launch(2);
   return launch_check();
 }
 

@@ -83,6 +83,20 @@ cudaError_t launch_prof_bucket(const Job &j, void *ws, const Layout &lo, uint32_
                                int64_t chunk, int64_t *cc, cudaStream_t st, int32_t *wsrc = nullptr,
                                uint32_t *crange = nullptr);
 constexpr int64_t kBucketTile = 16384;   // (jp_bucket.cu's tile: chunk ranges need chunk % kBucketTile == 0)
+// after launch_prof_bucket on the same workspace (its records still in place),
+// ADD_C: the last earlier writer of every raw read -> pred[i] (raw i only), and
+// three bitmaps of nw = ceil(n/32) words at bits (zeroed here): publish (the
+// writer is some raw read's pred), now (last writer of an address no exposed read
+// touches), later (last writer of an address that has an exposed read).
+// hdr[H_PRED_FAIL] > 0 if the pass could not hold some bucket's writers.
+cudaError_t launch_prof_pred(const Job &j, void *ws, const Layout &lo, int32_t *pred, uint32_t *bits,
+                             cudaStream_t st);
+// one-window on-chip TLS over a loop with WAR / WAW (path 9, reading B14): pred and
+// bits from launch_prof_pred, graw the profile's raw words, V one tagged shadow
+// slot per ITERATION (zeroed); the kernel exits at once if gate[H_PRED_FAIL] != 0.
+// stats as launch_tls_flow's (stats[3] violations, stats[1] lost warps)
+cudaError_t launch_tls_flow_waw(const Job &j, const uint32_t *graw, const int32_t *pred, const uint32_t *bits,
+                                unsigned long long *V, int64_t *stats, const int64_t *gate, cudaStream_t st);
 // src_bits (nullable): also the TLS guide's RAW-source words (raw_bits then holds its raw words)
 cudaError_t launch_prof_classify(const Job &j, void *ws, const Layout &lo, uint32_t *raw_bits,
                                  int64_t chunk, int64_t *chunk_counts, cudaStream_t st, uint32_t *src_bits = nullptr,

@@ -187,6 +187,169 @@ static cudaError_t run_flow(const Job &j, const uint32_t *graw, const uint32_t *
   return cudaLaunchCooperativeKernel((const void *)k_tls_flow<DT>, dim3(grid), dim3(kFlowT), args, 0, st);
 }
 
+// ---------------------------------------------------------------------------
+// Path 9 (reading B14): the same one window over a loop WITH WAR / WAW.  What
+// changes against path 8:
+//   recovery: the writer a violator must see is the LAST earlier writer of its
+//             address, pred(i) (the profile's last-writer pass records it), and
+//             its shadow slot is per ITERATION (V[pred]), since an address has
+//             several values over the loop;
+//   SE:       a non-violator's exposed read is of an element no earlier
+//             iteration writes -- but a later one may (WAR): nothing writes A
+//             in place except an address's last writer, and the last writer of
+//             an address that has such an exposed read waits for the window's
+//             one grid barrier (`later`); every other last writer (`now`)
+//             commits at once -- no exposed read of its address exists, and
+//             every other read of it is a violator fed from V;
+//   commit:   the final value of an address is its last writer's (WAW order),
+//             exactly the sequential state; writers that are not last only
+//             publish (if some violator reads them).
+// Statistics: jpo_sim_tls_fwd with W = n, as path 8.
+// ---------------------------------------------------------------------------
+struct FlowSetW {
+  int32_t r[kFlowK], w[kFlowK], pr[kFlowK];
+  uint32_t f[kFlowK];   // the iteration's bits: raw 1, publish 2, commit now 4, commit later 8
+  uint32_t x[kFlowK];
+};
+constexpr uint32_t kFRaw = 1, kFPub = 2, kFNow = 4, kFLater = 8;
+
+template <int DT>
+struct FlowW {
+  DLoop L;
+  const uint32_t *graw, *gpub, *gnow, *glater;
+  const int32_t *pred;
+  unsigned long long *V;
+  uint32_t G, g, n, io;
+  uint32_t viol = 0;
+  bool lost = false;
+
+  __device__ __forceinline__ bool act(uint32_t base, int k) const { return base + (uint32_t)k * G + g < n; }
+  __device__ __forceinline__ uint32_t it(uint32_t base, int k) const { return base + (uint32_t)k * G + g; }
+  __device__ __forceinline__ void load(uint32_t base, FlowSetW &s) const {
+#pragma unroll
+    for (int k = 0; k < kFlowK; k++) {
+      s.f[k] = 0;
+      if (!act(base, k)) continue;
+      const uint32_t i = it(base, k), q = i >> 5, sh = i & 31;
+      s.r[k] = L.r ? __ldcs(L.r + i) : (int32_t)(io + i);
+      s.w[k] = L.w ? __ldcs(L.w + i) : (int32_t)(io + i);
+      s.f[k] = ((__ldcs(graw + q) >> sh) & 1u) | ((__ldcs(gpub + q) >> sh) & 1u) << 1 |
+               ((__ldcs(gnow + q) >> sh) & 1u) << 2 | ((__ldcs(glater + q) >> sh) & 1u) << 3;
+    }
+#pragma unroll
+    for (int k = 0; k < kFlowK; k++)
+      if (s.f[k] & kFRaw) s.pr[k] = __ldcs(pred + it(base, k));
+  }
+  __device__ __forceinline__ void gather(uint32_t base, FlowSetW &s) const {
+#pragma unroll
+    for (int k = 0; k < kFlowK; k++)
+      if (act(base, k) && !(s.f[k] & kFRaw)) s.x[k] = __ldcg(L.A + s.r[k]);
+  }
+  __device__ __forceinline__ void commit(const FlowSetW &s, uint32_t base, int k, uint32_t v) const {
+    if (s.f[k] & kFNow) __stcg(L.A + s.w[k], v);
+    if (s.f[k] & (kFPub | kFLater))
+      asm volatile("st.relaxed.gpu.global.u64 [%0], %1;" ::"l"(V + it(base, k)), "l"(kFlowTag | v) : "memory");
+  }
+  __device__ __forceinline__ void run(uint32_t base, FlowSetW &s) {
+    uint32_t pend = 0;
+#pragma unroll
+    for (int k = 0; k < kFlowK; k++) {
+      if (!act(base, k)) continue;
+      if (s.f[k] & kFRaw) pend |= 1u << k;
+      else commit(s, base, k, op_add<DT>(s.x[k], L.c0));
+    }
+    viol += __popc(pend);
+    long long spins = 0;
+    while (__any_sync(0xffffffffu, pend)) {
+#pragma unroll
+      for (int k = 0; k < kFlowK; k++) {
+        if ((pend >> k) & 1u) {
+          unsigned long long v;
+          asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(v) : "l"(V + s.pr[k]) : "memory");
+          if ((v >> 32) == 1ull) {
+            commit(s, base, k, op_add<DT>((uint32_t)v, L.c0));
+            pend &= ~(1u << k);
+          }
+        }
+      }
+      if (++spins > kFlowSpinLimit) {
+        lost = lost || pend;
+        break;
+      }
+    }
+  }
+};
+
+template <int DT>
+__global__ void __launch_bounds__(kFlowT, JP_FLOW_MINB) k_tls_flow_waw(DLoop L, const uint32_t *graw, const int32_t *pred,
+                                                           const uint32_t *bits, unsigned long long *V,
+                                                           int64_t *stats, const int64_t *gate) {
+  if (gate && gate[H_PRED_FAIL] != 0) return;   // grid-uniform: no barrier is entered
+  const uint32_t nw = (uint32_t)((L.n + 31) / 32);
+  FlowW<DT> F;
+  F.L = L; F.graw = graw; F.pred = pred; F.V = V;
+  F.gpub = bits; F.gnow = bits + nw; F.glater = bits + 2 * nw;
+  F.G = gridDim.x * (uint32_t)kFlowT;
+  F.g = blockIdx.x * (uint32_t)kFlowT + threadIdx.x;
+  F.n = (uint32_t)L.n;
+  F.io = (uint32_t)L.ioff;
+  const uint32_t step = F.G * (uint32_t)kFlowK;
+  FlowSetW a, b;
+  F.load(0, a);
+  F.gather(0, a);
+  for (uint32_t base = 0; base < F.n; base += 2 * step) {
+    if (base + step < F.n) { F.load(base + step, b); F.gather(base + step, b); }
+    F.run(base, a);
+    if (base + step >= F.n) break;
+    if (base + 2 * step < F.n) { F.load(base + 2 * step, a); F.gather(base + 2 * step, a); }
+    F.run(base + step, b);
+  }
+  const uint32_t v = __reduce_add_sync(0xffffffffu, F.viol);
+  const unsigned lost = __any_sync(0xffffffffu, F.lost);
+  if ((threadIdx.x & 31) == 0) {
+    if (v) atomicAdd(reinterpret_cast<unsigned long long *>(&stats[3]), (unsigned long long)v);
+    if (lost) atomicAdd(reinterpret_cast<unsigned long long *>(&stats[1]), 1ull);
+  }
+  // the window's one barrier: then the last writers whose address had an exposed
+  // read (its window-start value is no longer needed) commit from their slots
+  cg::this_grid().sync();
+  for (uint32_t q = F.g; q < nw; q += F.G) {
+    uint32_t m = __ldcs(F.glater + q);
+    while (m) {
+      const uint32_t i = q * 32 + (uint32_t)__ffs(m) - 1;
+      m &= m - 1;
+      const int32_t wi = L.w ? L.w[i] : (int32_t)(F.io + i);
+      L.A[wi] = (uint32_t)__ldcg(V + i);
+    }
+  }
+}
+
+template <int DT>
+static cudaError_t run_flow_waw(const Job &j, const uint32_t *graw, const int32_t *pred, const uint32_t *bits,
+                                unsigned long long *V, int64_t *stats, const int64_t *gate, cudaStream_t st) {
+  int maxb = 0;
+  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&maxb, (const void *)k_tls_flow_waw<DT>, kFlowT, 0);
+  if (maxb < 1) return cudaErrorInvalidConfiguration;
+  int grid = num_sms() * maxb;
+  const int64_t need = (j.d.n + kFlowT - 1) / kFlowT;
+  if (need < grid) grid = (int)(need < 1 ? 1 : need);
+  DLoop d = j.d;
+  void *args[] = {&d, &graw, &pred, &bits, &V, &stats, &gate};
+  note_launch();
+  return cudaLaunchCooperativeKernel((const void *)k_tls_flow_waw<DT>, dim3(grid), dim3(kFlowT), args, 0, st);
+}
+
+cudaError_t launch_tls_flow_waw(const Job &j, const uint32_t *graw, const int32_t *pred, const uint32_t *bits,
+                                unsigned long long *V, int64_t *stats, const int64_t *gate, cudaStream_t st) {
+  cudaMemsetAsync(stats, 0, 4 * sizeof(int64_t), st);
+  if (j.d.n == 0) return launch_check();
+  if (j.op != JP_OP_ADD_C) return cudaErrorInvalidValue;
+  cudaError_t e = j.dt == JP_F32 ? run_flow_waw<JP_F32>(j, graw, pred, bits, V, stats, gate, st)
+                                 : run_flow_waw<JP_I32>(j, graw, pred, bits, V, stats, gate, st);
+  if (e != cudaSuccess) return e;
+  return launch_check();
+}
+
 // Device stats after the kernel: stats[3] = violations (raw iterations),
 // stats[1] = number of warps that gave up waiting for a writer (0 unless the
 // guide was inconsistent); the caller turns them into jpo_sim_tls_fwd's

@@ -137,14 +137,15 @@ def test_doall_indirect_multi_trip(op, dt, generic, monkeypatch):
 @pytest.mark.parametrize("d,delta", [(0.01, 1024), (0.10, 1024), (0.01, 1 << 20), (0.10, 1 << 20)])
 def test_config3_waw_full_size_restart(d, delta):
     """Config 3's shape with write-after-write (on-chip recovery illegal), N = 2^24,
-    through jp_schedule -- the bench's config3_waw rows: restart TLS under the
-    distance-steered cap; every byte of A and the statistics of jpo_sim_tls under
-    that cap."""
+    through jp_schedule with tls_recovery = 1 -- the bench's config3_waw restart
+    rows: restart TLS under the distance-steered cap; every byte of A and the
+    statistics of jpo_sim_tls under that cap (the default call runs path 9,
+    tests/test_gpu_flow_waw.py)."""
     wl = synth.config3_waw(d, delta=delta)
     ref = to_oracle(wl)
     g = wl.to(DEV)
     L = jp.Loop.from_workload(g)
-    res = jp.jp_schedule(L, jp.workspace(L))
+    res = jp.jp_schedule(L, jp.workspace(L), tls_recovery=1)
     torch.cuda.synchronize()
     assert res["mode"] == jp.JP_MODE_TLS and res["tls_recovery"] == jp.JP_TLS_RESTART, res
     p = O.profile(ref)
