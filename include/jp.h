@@ -151,8 +151,11 @@ typedef struct {
                                    density: clamp(pow2ceil(sqrt(1000/d_raw)), 256, 1024)
                                    (measured optimum of the single-CTA path)      */
   int32_t tls_recovery;         /* 0 auto (JP_TLS_ONCHIP when the profile shows
-                                   waw_iters == 0, else JP_TLS_RESTART), 1 restart,
-                                   2 on-chip.  With tls_path 0 and tls_recovery 0
+                                   waw_iters == 0, else JP_TLS_RESTART -- except
+                                   that jp_schedule runs an ADD_C loop with
+                                   WAR / WAW profiled by address buckets on path
+                                   9 when its last-writer pass holds the loop),
+                                   1 restart, 2 on-chip.  With tls_path 0 and tls_recovery 0
                                    a SEQ_RECOMMENDED loop (mode C) runs on the
                                    one-warp program-order path 7              */
   int32_t static_check;         /* 0: before profiling, (a) structural RAW-freedom
@@ -178,10 +181,23 @@ typedef struct {
   int32_t tls_path;             /* TLS: jp_tls_cfg.path that ran (1, 2, 3; 4 tiny
                                    one-CTA schedule; 5 / 6 on-chip recovery on a
                                    cluster / on every SM; 7 one-warp program order
-                                   for mode C; 8 on-chip recovery in one window)  */
+                                   for mode C; 8 on-chip recovery in one window;
+                                   9 the same over a loop with WAR / WAW
+                                   (reading B14, jp_schedule only: every
+                                   violator fed from the LAST earlier writer of
+                                   its address, from a per-iteration shadow slot
+                                   in region 8, its index in region 7; last
+                                   writers commit at once, or after the window's
+                                   one grid barrier when an exposed read of
+                                   their address needs the window-start value;
+                                   stats as path 8: one window, violations =
+                                   raw iterations, jpo_sim_tls_fwd with W = n;
+                                   an address with > 4096 writers, or a bucket
+                                   of 8192 addresses with > ~49K writes, keeps
+                                   the windowed paths))  */
   int32_t tls_guided;           /* TLS: 1 when the guide (jp_tls_guide) steered it    */
   int32_t tls_recovery;         /* TLS: jp_tls_recovery that ran                      */
-  int32_t tls_cluster;          /* TLS: CTAs of the cluster (paths 3, 5) or grid (6, 8) */
+  int32_t tls_cluster;          /* TLS: CTAs of the cluster (paths 3, 5) or grid (6, 8, 9) */
 } jp_sched_result;
 
 /* ---- workspace -------------------------------------------------------------

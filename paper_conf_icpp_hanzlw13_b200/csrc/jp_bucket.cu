@@ -441,9 +441,8 @@ struct PredOut {
 };
 
 template <bool BIG>
-__global__ void __launch_bounds__(BIG ? 1024 : 512, BIG ? 1 : 2) k_bk_pred(BkView V, const uint32_t *base,
-                                                                           const uint32_t *tot,
-                                                                           const unsigned long long *rec, PredOut O) {
+__device__ __forceinline__ void pred_bucket(int b, const uint32_t *base, const uint32_t *tot,
+                                            const unsigned long long *rec, const PredOut &O) {
   constexpr int kT = BIG ? 1024 : 512;
   constexpr uint32_t kCap = BIG ? kPredCapB : kPredCapS;
   extern __shared__ uint32_t s_dyn[];
@@ -454,8 +453,6 @@ __global__ void __launch_bounds__(BIG ? 1024 : 512, BIG ? 1 : 2) k_bk_pred(BkVie
   uint32_t *wl = xflag + kBSpan / 32;       // [kCap] writer lists
   __shared__ uint32_t s_wsum[kT / 32];
   __shared__ uint32_t s_nw;
-  const int b = blockIdx.x;
-  if (BIG && !O.redo[b]) return;
   const uint32_t total = tot[b];
   const unsigned long long *rb = rec + base[b];
   for (int k = threadIdx.x; k < kBSpan; k += kT) cur[k] = 0;
@@ -548,6 +545,20 @@ __global__ void __launch_bounds__(BIG ? 1024 : 512, BIG ? 1 : 2) k_bk_pred(BkVie
     for (uint32_t p = p0 + 1; p < p1; p++) last = max(last, wl[p]);
     uint32_t *bits = (xflag[al >> 5] >> (al & 31)) & 1u ? O.later : O.now;
     atomicOr(&bits[last >> 5], 1u << (last & 31));
+  }
+}
+
+__global__ void __launch_bounds__(512, 2) k_bk_pred(const uint32_t *base, const uint32_t *tot,
+                                                    const unsigned long long *rec, PredOut O) {
+  pred_bucket<false>(blockIdx.x, base, tot, rec, O);
+}
+// the big tier: one CTA per SM walks the buckets and redoes the marked ones
+__global__ void __launch_bounds__(1024, 1) k_bk_pred_big(int B, const uint32_t *base, const uint32_t *tot,
+                                                         const unsigned long long *rec, PredOut O) {
+  for (int b = blockIdx.x; b < B; b += gridDim.x) {
+    if (!O.redo[b]) continue;
+    pred_bucket<true>(b, base, tot, rec, O);
+    __syncthreads();   // (shared memory reused by the next bucket)
   }
 }
 
@@ -672,13 +683,13 @@ cudaError_t launch_prof_pred(const Job &j, void *ws, const Layout &lo, int32_t *
   // redo flags in the per-tile offsets (P.cnt: the scatter was their last reader)
   if (e == cudaSuccess) e = cudaMemsetAsync(P.cnt, 0, 4 * (size_t)P.v.B, st);
   if (e == cudaSuccess)
-    e = cudaFuncSetAttribute(k_bk_pred<false>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)kPredSmemS);
+    e = cudaFuncSetAttribute(k_bk_pred, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)kPredSmemS);
   if (e == cudaSuccess)
-    e = cudaFuncSetAttribute(k_bk_pred<true>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)kPredSmemB);
+    e = cudaFuncSetAttribute(k_bk_pred_big, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)kPredSmemB);
   if (e != cudaSuccess) return e;
   PredOut O{pred, bits, bits + nw, bits + 2 * nw, at<int64_t>(ws, lo, R_HEADER), P.cnt};
-  k_bk_pred<false><<<P.v.B, 512, kPredSmemS, st>>>(P.v, P.base, P.tot, P.rec, O);
-  k_bk_pred<true><<<P.v.B, 1024, kPredSmemB, st>>>(P.v, P.base, P.tot, P.rec, O);
+  k_bk_pred<<<P.v.B, 512, kPredSmemS, st>>>(P.base, P.tot, P.rec, O);
+  k_bk_pred_big<<<std::min(P.v.B, num_sms()), 1024, kPredSmemB, st>>>(P.v.B, P.base, P.tot, P.rec, O);
   note_launch(2);
   return launch_check();
 }
