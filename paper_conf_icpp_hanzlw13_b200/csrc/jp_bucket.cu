@@ -49,7 +49,10 @@ constexpr int kMaxBuckets = 8192;           // len_A <= 2^26
 constexpr int kMaxTiles = 16384;            // n <= 2^26
 constexpr int kSmemChunks = 1024;           // per-chunk counts kept in shared memory up to this many chunks
 // record (8 bytes): local iteration (low word) | address in the bucket << 32 | write << 63
-constexpr unsigned long long kRecW = 1ull << 63;
+// | also-read << 62: an ADD_C iteration whose read and write are the same address
+// (an in-place update, A[w[i]] = A[w[i]] + c) files ONE record for both accesses
+constexpr unsigned long long kRecW = 1ull << 63, kRecRW = 1ull << 62;
+__device__ __forceinline__ bool rec_reads(unsigned long long x) { return !(x & kRecW) || (x & kRecRW); }
 
 struct BkView {
   const int32_t *r, *w;   // ADD_C: read r, write w; SAXPY: w only (NULL => identity ioff + i)
@@ -127,7 +130,7 @@ __global__ void __launch_bounds__(kBThreads) k_bk_count(BkView V, int vec, uint3
           const uint32_t c = (uint32_t)q4(r4, k);
           const bool okc = c < V.lenA;
           nbad += !okc;
-          atomicAdd(&h[okc ? c >> kBShift : 0], 1u);
+          if (c != a) atomicAdd(&h[okc ? c >> kBShift : 0], 1u);   // (c == a: one record for both)
           if (okc) { mn = min(mn, c); mx = max(mx, c); }
         }
       }
@@ -261,18 +264,25 @@ __global__ void __launch_bounds__(kBThreads) k_bk_scatter(BkView V, int vec, con
       a[OP == JP_OP_ADD_C ? 2 * k : k] = (uint32_t)q4(w4, k);
       if constexpr (OP == JP_OP_ADD_C) a[2 * k + 1] = (uint32_t)q4(r4, k);
     }
+    // an iteration reading the address it writes: one record (write | also-read)
+    bool same[4];
+#pragma unroll
+    for (int k = 0; k < 4; k++) same[k] = OP == JP_OP_ADD_C && a[2 * k] == a[2 * k + 1];
 #pragma unroll
     for (int m = 0; m < kA; m++) {
       if (a[m] >= V.lenA) a[m] = 0;   // (the count pass filed it under bucket 0 too)
       const int k = OP == JP_OP_ADD_C ? m >> 1 : m;
-      pos[m] = k < kn ? atomicAdd(&cur[a[m] >> kBShift], 1u) : 0u;
+      const bool skip = OP == JP_OP_ADD_C && (m & 1) && same[k];
+      pos[m] = k < kn && !skip ? atomicAdd(&cur[a[m] >> kBShift], 1u) : 0u;
     }
 #pragma unroll
     for (int m = 0; m < kA; m++) {
       const int k = OP == JP_OP_ADD_C ? m >> 1 : m;
       const bool wr = OP == JP_OP_ADD_C ? (m & 1) == 0 : true;
-      if (k < kn) {
-        stage[pos[m]] = (uint32_t)(il0 + k) | (a[m] & (kBSpan - 1)) << kTShift | (wr ? 1u << 31 : 0u);
+      const bool skip = OP == JP_OP_ADD_C && (m & 1) && same[k];
+      if (k < kn && !skip) {
+        stage[pos[m]] = (uint32_t)(il0 + k) | (a[m] & (kBSpan - 1)) << kTShift | (wr ? 1u << 31 : 0u) |
+                        (wr && same[k] ? 1u << 30 : 0u);
         stb[pos[m]] = (uint16_t)(a[m] >> kBShift);
       }
     }
@@ -286,7 +296,8 @@ __global__ void __launch_bounds__(kBThreads) k_bk_scatter(BkView V, int vec, con
   for (uint32_t k = threadIdx.x; k < nrec; k += kBThreads) {
     const uint32_t x = stage[k];
     rec[k + gpos[stb[k]]] = (unsigned long long)(i0 + (x & (kTile - 1))) |
-                            (unsigned long long)((x >> kTShift) & (kBSpan - 1)) << 32 | (x >> 31 ? kRecW : 0ull);
+                            (unsigned long long)((x >> kTShift) & (kBSpan - 1)) << 32 | (x >> 31 ? kRecW : 0ull) |
+                            ((x >> 30) & 1u ? kRecRW : 0ull);
   }
 }
 
@@ -342,7 +353,8 @@ __global__ void __launch_bounds__(kEvalThreads) k_bk_eval(BkView V, const uint32
   sweep([&](unsigned long long x) {
     const uint32_t i = (uint32_t)x, al = (uint32_t)(x >> 32) & (kBSpan - 1);
     if (x & kRecW) atomicMin(&minW[al], i);
-    else if constexpr (OP == JP_OP_ADD_C) atomicMin(&minR[al], i);
+    if constexpr (OP == JP_OP_ADD_C)
+      if (rec_reads(x)) atomicMin(&minR[al], i);
   });
   __syncthreads();
   // pass 2: every access against the final tables
@@ -354,14 +366,14 @@ __global__ void __launch_bounds__(kEvalThreads) k_bk_eval(BkView V, const uint32
     bool raw, war = false, waw = false;
     if (x & kRecW) {
       waw = jw < i;
-      war = (OP == JP_OP_ADD_C ? minR[al] : jw) < i;
-      raw = OP == JP_OP_SAXPY && waw;
+      war = (OP == JP_OP_ADD_C ? minR[al] : jw) < i;   // (an also-read record's own read is minR = i: not < i)
+      raw = OP == JP_OP_SAXPY ? waw : (x & kRecRW) && waw;
     } else {
       raw = jw < i;
     }
     c_raw += raw; c_war += war; c_waw += waw;
     if (raw) {
-      if (O.wsrc && !(x & kRecW)) O.wsrc[i] = (int32_t)jw;
+      if (O.wsrc && rec_reads(x)) O.wsrc[i] = (int32_t)jw;
       if (O.graw) atomicOr(&O.graw[i >> 5], 1u << (i & 31));
       if (O.gsrc) atomicOr(&O.gsrc[jw >> 5], 1u << (jw & 31));
       atomicAdd(&s_dist[31 - __clz(i - jw)], 1u);
@@ -520,7 +532,7 @@ __device__ __forceinline__ void pred_bucket(int b, const uint32_t *base, const u
   __syncthreads();
   // reads: the largest writer below i in the address's list
   sweep([&](unsigned long long x) {
-    if (x & kRecW) return;
+    if (!rec_reads(x)) return;
     const uint32_t i = (uint32_t)x, al = (uint32_t)(x >> 32) & (kBSpan - 1);
     const uint32_t p0 = al ? cur[al - 1] : 0u, p1 = cur[al];
     if (p0 == p1) return;   // an address nobody writes
