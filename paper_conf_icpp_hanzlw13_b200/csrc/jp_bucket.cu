@@ -81,12 +81,11 @@ __device__ __forceinline__ int q4(const int4 &v, int k) { return k == 0 ? v.x : 
 // Visit the accesses of tile blockIdx.x four iterations at a time (16-byte
 // index loads, kU quads in flight per lane): f(a[8], wr[8], il0, kn) gets the
 // quad's accesses -- ADD_C: (w, r) of each of the kn <= 4 iterations, SAXPY: w.
-template <int OP, typename F>
+template <int OP, int kU = 4, typename F>
 __device__ __forceinline__ void for_tile(const BkView &V, bool vec, F &&f) {
   const int64_t t0 = (int64_t)blockIdx.x << kTShift;
   const int64_t tn = V.n - t0 < kTile ? V.n - t0 : kTile;
   const int nq = (int)((tn + 3) >> 2);
-  constexpr int kU = 4;
   for (int q0 = threadIdx.x; q0 < nq; q0 += kBThreads * kU) {
     int4 vw[kU], vr[kU];
 #pragma unroll
@@ -109,7 +108,7 @@ __device__ __forceinline__ void for_tile(const BkView &V, bool vec, F &&f) {
 
 // cnt[t * B + b] = accesses of tile t into bucket b; out-of-range indices counted into *bad
 template <int OP>
-__global__ void __launch_bounds__(kBThreads) k_bk_count(BkView V, int vec, uint32_t *cnt, int64_t *bad) {
+__global__ void __launch_bounds__(kBThreads, 2) k_bk_count(BkView V, int vec, uint32_t *cnt, int64_t *bad) {
   extern __shared__ uint32_t h[];
   for (int b = threadIdx.x; b < V.B; b += kBThreads) h[b] = 0;
   __syncthreads();
@@ -117,7 +116,8 @@ __global__ void __launch_bounds__(kBThreads) k_bk_count(BkView V, int vec, uint3
   uint32_t mn = 0xFFFFFFFFu, mx = 0u;   // the tile's address range (crange: a tile lies in one chunk)
   // an out-of-range index is counted (the profile then fails) and filed under
   // bucket 0, consistently with the scatter below
-  for_tile<OP>(V, vec, [&](const int4 &w4, const int4 &r4, int, int kn) {
+  // (two quads in flight per lane: 32 registers, two CTAs per SM)
+  for_tile<OP, 2>(V, vec, [&](const int4 &w4, const int4 &r4, int, int kn) {
 #pragma unroll
     for (int k = 0; k < 4; k++) {
       if (k < kn) {
