@@ -399,7 +399,8 @@ int32_t jp_select_mode(const jp_loop *L, const jp_profile *p, double tau_high) {
 // after_sample (nullable): called right after the prefix sample is launched,
 // before the host waits for it (jp_schedule queues side-stream work there)
 static jp_status static_check(const jp_loop *L, const Job &j, void *ws, const Layout &lo, jp_static *out,
-                              cudaStream_t st, const std::function<void()> *after_sample = nullptr) {
+                              cudaStream_t st, const std::function<void()> *after_sample = nullptr,
+                              bool skip_prefix = false) {
   bool kicked = false;
   auto kick = [&]() {
     if (after_sample && !kicked) (*after_sample)();
@@ -408,7 +409,7 @@ static jp_status static_check(const jp_loop *L, const Job &j, void *ws, const La
   memset(out, 0, sizeof *out);
   int64_t *hdr = at<int64_t>(ws, lo, R_HEADER);
   int *flags = reinterpret_cast<int *>(&hdr[H_AFFINE]);
-  {
+  if (!skip_prefix) {
     // a 64-entry prefix of each index array first: an array that is not affine
     // there is not affine at all, and the full pass (a read of every index
     // array) is skipped -- the common case of indirect loops
@@ -820,7 +821,7 @@ static jp_status run_tls_job(const jp_loop *L, const Job &j, const jp_tls_cfg *c
     JP_CUDA(launch_tls_fwd(j, tp.window, tp.cluster, bits, bsrc, &hdr[H_TLS_COMMITTED], st), "tls on-chip");
   } else if (tp.path == 8) {
     auto *V = at<unsigned long long>(ws, lo, R_TLS_C_A);
-    if (!(s_clean & 2)) cudaMemsetAsync(V, 0, 8 * (size_t)L->len_A, st);   // no shadow value yet
+    if (!(s_clean & 6)) cudaMemsetAsync(V, 0, 8 * (size_t)L->len_A, st);   // no shadow value yet
     JP_CUDA(launch_tls_flow(j, bits, bsrc, V, &hdr[H_TLS_COMMITTED], st), "tls one window");
   } else if (tp.path == 6) {
     auto *S = at<unsigned long long>(ws, lo, R_TLS_S_A);
@@ -1368,30 +1369,18 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
   // (the write log of paths 5 / 6, unused by path 8)
   int32_t *wsrc = nullptr;
   uint32_t *crange = nullptr;   // per-chunk address ranges from the bucket profile (task PDG prefilter)
-  cudaEvent_t vev = nullptr;    // side-stream clear of the shadow values; every exit orders st after it
-  struct JoinVev {
-    cudaEvent_t &e; cudaStream_t s;
-    void join() { if (e) { cudaStreamWaitEvent(s, e, 0); cudaEventDestroy(e); e = nullptr; } }
-    ~JoinVev() { join(); }
-  } join_vev{vev, st};
+  unsigned long long *vclr = nullptr;   // the shadow values, cleared where path 8 polls them by the profile
   if (bucket_profile_ok(j, ws, lo)) {   // large A: the profile by address buckets (jp_bucket.cu)
     s_fresh = false;                    // (region 7 is not filled: the TLS task resets it)
     if (gbits && j.op == JP_OP_ADD_C && lo.bytes[R_TLS_S_A] >= 4 * (size_t)L->n && !getenv("JP_TLS_NO_FLOW"))
       wsrc = at<int32_t>(ws, lo, R_TLS_S_A);
     if (chunk % kBucketTile == 0 && !getenv("JP_TASK_MASKS_ALWAYS"))
       crange = reinterpret_cast<uint32_t *>(sch + sl.crange);
-    // the shadow values of a one-window TLS task start at zero: cleared on a
-    // side stream while the profile runs
-    auto *V = at<unsigned long long>(ws, lo, R_TLS_C_A);
-    if (wsrc && V && cudaEventCreateWithFlags(&vev, cudaEventDisableTiming) == cudaSuccess) {
-      cudaStream_t side = g_pool.get(40);
-      cudaEventRecord(vev, st);
-      cudaStreamWaitEvent(side, vev, 0);
-      cudaMemsetAsync(V, 0, lo.bytes[R_TLS_C_A], side);
-      cudaEventRecord(vev, side);
-    }
+    // the shadow slots a one-window TLS task polls (V at every raw read's
+    // address) are cleared by the profile itself
+    vclr = wsrc ? at<unsigned long long>(ws, lo, R_TLS_C_A) : nullptr;
     JP_CUDA(launch_prof_bucket(j, ws, lo, gbits, gbits ? gbits + (L->n + 31) / 32 : nullptr, chunk, cc, st, wsrc,
-                               crange),
+                               crange, vclr),
             "profile (buckets)");
   } else {
     JP_CUDA(launch_prof_stamp(j, ws, lo, st, pairs), "profile stamp");
@@ -1458,9 +1447,7 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
   std::vector<int> flow_tasks;  // ... of them, run as one window (path 8): stats completed on the host
   // the side-stream clear (done long before: it overlapped the profile) is
   // joined before any task runs
-  const bool v_zeroed_side = vev != nullptr;
-  join_vev.join();
-  bool v_zeroed = v_zeroed_side;
+  bool v_zeroed = vclr != nullptr;
   cudaEvent_t ev0;
   JP_CUDA(cudaEventCreateWithFlags(&ev0, cudaEventDisableTiming), "event");
   std::vector<cudaEvent_t> evs;
@@ -1884,7 +1871,8 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
   // it: the clear would hold every SM while the host waits for the sample), so
   // it overlaps the sample's round trip and the profile
   const std::function<void()> clear_v = [&]() {
-    if (!(gfuse && (pairs || bucket)) || vdone) return;
+    // (the bucket profile clears the slots path 8 uses itself: V[a] = 0 at every raw read's address)
+    if (!(gfuse && pairs) || vdone) return;
     auto *V = at<unsigned long long>(ws, lg, R_TLS_C_A);
     if (V && cudaEventCreateWithFlags(&vdone, cudaEventDisableTiming) == cudaSuccess) {
       cudaStream_t side = g_pool.get(40);
@@ -1894,7 +1882,12 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
       cudaEventRecord(vdone, side);
     }
   };
-  if (c.static_check == 0 && ws) {
+  // with the address-bucket profile the static check's affine sample rides on
+  // the profile's first kernel (the rest of the profile exits when the sample
+  // looks affine): no host round trip before the profile starts
+  const bool defer_static = c.static_check == 0 && ws && bucket && tiny_mirror().host && L->n >= 3 &&
+                            !getenv("JP_NO_DEFER_STATIC");
+  if (c.static_check == 0 && ws && !defer_static) {
     // static analysis lite: affine, in-range, conflict-free -> DOALL without a profile
     Layout ls;
     if (jp_status e0 = check_ws(L, ws, ws_bytes, 0, ls)) { join_fill(); return e0; }
@@ -1928,7 +1921,43 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
     if (bucket) {
       // large A: the profile by address buckets (jp_bucket.cu), guide words included
       uint32_t *g = at<uint32_t>(ws, lg, R_GUIDE);
-      JP_CUDA(launch_prof_bucket(j, ws, lg, g, g + (L->n + 31) / 32, 0, nullptr, st), "profile (buckets)");
+      TinyMirror &mm = tiny_mirror();
+      const unsigned long long seq = defer_static ? ++mm.seq : 0;
+      JP_CUDA(launch_prof_bucket(j, ws, lg, g, g + (L->n + 31) / 32, 0, nullptr, st, nullptr, nullptr,
+                                 at<unsigned long long>(ws, lg, R_TLS_C_A), defer_static ? (int)std::min<int64_t>(L->n, 64) : 0,
+                                 defer_static ? reinterpret_cast<long long *>(mm.dev + 19) : nullptr, seq),
+              "profile (buckets)");
+      clean |= 4;   // V clear at every address path 8 polls
+      if (defer_static) {
+        volatile unsigned long long *flag = reinterpret_cast<volatile unsigned long long *>(&mm.host[20]);
+        for (unsigned spins = 0; *flag != seq; spins++) {
+          if ((spins & 1023) == 1023) {
+            const cudaError_t q = cudaStreamQuery(st);
+            if (q != cudaSuccess && q != cudaErrorNotReady) return cuda_fail(q, "profile");
+            if (q == cudaSuccess && *flag != seq) return fail(JP_ERR_CUDA, "profile did not publish its affine sample");
+          }
+        }
+        if (*reinterpret_cast<volatile int64_t *>(&mm.host[19]) != 0) {
+          // the sample looks affine (the profile's kernels exited): the full static
+          // check, then DOALL or the profile proper
+          Layout ls;
+          JP_TRY(check_ws(L, ws, ws_bytes, 0, ls));
+          jp_static sa;
+          JP_TRY(static_check(L, j, ws, ls, &sa, st, nullptr, true));
+          if (sa.independent && sa.in_range) {
+            res->mode = JP_MODE_DOALL;
+            res->profiled = 0;
+            res->n_tasks = 1;
+            res->n_batches = 1;
+            JP_CUDA(launch_doall(j, st), "doall");
+            res->task_mode_iters[JP_MODE_DOALL] = L->n;
+            return JP_OK;
+          }
+          JP_CUDA(launch_prof_bucket(j, ws, lg, g, g + (L->n + 31) / 32, 0, nullptr, st, nullptr, nullptr,
+                                     at<unsigned long long>(ws, lg, R_TLS_C_A)),
+                  "profile (buckets)");
+        }
+      }
     } else {
       if (pairs) JP_CUDA(launch_prof_stamp(j, ws, lg, st, true, pairs_ready), "profile stamp");
       else JP_TRY(jp_profile_stamp(L, ws, ws_bytes, stp));
@@ -1943,7 +1972,7 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
     // mode B with war = waw = 0 -- exactly when run_mode below would pick path 8
     // -- so the GPU does not idle through the header's round trip; the header
     // travels to the host on a side stream meanwhile.
-    spec = vclear && j.op == JP_OP_ADD_C && c.tls_path == 0 && c.tls_window == 0 && c.tls_recovery != 1 &&
+    spec = (vclear || bucket) && j.op == JP_OP_ADD_C && c.tls_path == 0 && c.tls_window == 0 && c.tls_recovery != 1 &&
            L->n > 0 && !getenv("JP_TLS_NO_FLOW") && !getenv("JP_NO_SPEC_FLOW");
     cudaEvent_t ep = nullptr, ec = nullptr;
     if (spec && (cudaEventCreateWithFlags(&ep, cudaEventDisableTiming) != cudaSuccess ||
@@ -2024,8 +2053,7 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
     auto *bits = reinterpret_cast<uint32_t *>(pred + ((L->n + 63) & ~(int64_t)63));
     auto *V = at<unsigned long long>(ws, lg, R_TLS_C_A);
     const uint32_t *graw = at<uint32_t>(ws, lg, R_GUIDE);
-    if (!(clean & 2)) JP_CUDA(cudaMemsetAsync(V, 0, 8 * (size_t)L->n, st), "shadow clear");
-    JP_CUDA(launch_prof_pred(j, ws, lg, pred, bits, st), "last writers");
+    JP_CUDA(launch_prof_pred(j, ws, lg, pred, bits, V, st), "last writers");   // (clears V[pred])
     JP_CUDA(launch_tls_flow_waw(j, graw, pred, bits, V, &hd[H_TLS_COMMITTED], hd, st), "tls one window (waw)");
     int64_t h2[H_PRED_SEG + 1];
     JP_CUDA(d2h_small_sync(h2, hd, sizeof h2, st), "tls D2H");

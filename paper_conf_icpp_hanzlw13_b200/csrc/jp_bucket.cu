@@ -61,7 +61,9 @@ struct BkView {
   int B, T;
   uint32_t *crange;       // nullable: per chunk min / max address (chunk = ctiles tiles)
   int ctiles;
+  const int64_t *gate;    // nullable: the header's H_GATE word -- every kernel exits when it is nonzero
 };
+__device__ __forceinline__ bool gated(const int64_t *g) { return g && *(volatile const int64_t *)g != 0; }
 
 __device__ __forceinline__ int4 ld_idx4(const int32_t *p, int64_t i, int64_t n, int64_t ioff, bool vec) {
   if (!p) {
@@ -109,6 +111,7 @@ __device__ __forceinline__ void for_tile(const BkView &V, bool vec, F &&f) {
 // cnt[t * B + b] = accesses of tile t into bucket b; out-of-range indices counted into *bad
 template <int OP>
 __global__ void __launch_bounds__(kBThreads, 2) k_bk_count(BkView V, int vec, uint32_t *cnt, int64_t *bad) {
+  if (gated(V.gate)) return;
   extern __shared__ uint32_t h[];
   for (int b = threadIdx.x; b < V.B; b += kBThreads) h[b] = 0;
   __syncthreads();
@@ -154,7 +157,9 @@ __global__ void __launch_bounds__(kBThreads, 2) k_bk_count(BkView V, int vec, ui
 
 // per bucket: exclusive prefix over the tiles (in place) and the bucket total.
 // Block = 32 buckets (one per lane) x 32 tile segments (one per warp).
-__global__ void __launch_bounds__(1024) k_bk_scan_tiles(uint32_t *cnt, int T, int B, uint32_t *tot) {
+__global__ void __launch_bounds__(1024) k_bk_scan_tiles(uint32_t *cnt, int T, int B, uint32_t *tot,
+                                                         const int64_t *gate) {
+  if (gated(gate)) return;
   __shared__ uint32_t part[32][33];
   const int lane = threadIdx.x & 31, seg = threadIdx.x >> 5;
   const int b = blockIdx.x * 32 + lane;
@@ -179,7 +184,9 @@ __global__ void __launch_bounds__(1024) k_bk_scan_tiles(uint32_t *cnt, int T, in
 }
 
 // base[b] = exclusive prefix of tot over the buckets (one CTA)
-__global__ void __launch_bounds__(1024) k_bk_scan_buckets(const uint32_t *tot, int B, uint32_t *base) {
+__global__ void __launch_bounds__(1024) k_bk_scan_buckets(const uint32_t *tot, int B, uint32_t *base,
+                                                           const int64_t *gate) {
+  if (gated(gate)) return;
   __shared__ uint32_t ws[32];
   const int per = (B + 1023) / 1024, b0 = threadIdx.x * per;
   uint32_t s = 0;
@@ -213,6 +220,7 @@ __global__ void __launch_bounds__(1024) k_bk_scan_buckets(const uint32_t *tot, i
 template <int OP>
 __global__ void __launch_bounds__(kBThreads) k_bk_scatter(BkView V, int vec, const uint32_t *off, const uint32_t *tot,
                                                          const uint32_t *base, unsigned long long *rec) {
+  if (gated(V.gate)) return;
   // staging: 6 bytes per record -- il | address in the bucket << 14 | write << 31,
   // and the bucket (16 bits) -- so that a 16384-iteration tile fits one SM
   extern __shared__ uint32_t sm32[];
@@ -308,11 +316,14 @@ struct BkOut {
   int64_t *cc;
   int64_t gbase;              // global id of local iteration 0
   int32_t *wsrc;              // nullable: wsrc[i] = the first writer of raw iteration i's read (ADD_C)
+  unsigned long long *vclr;   // nullable: V[a] = 0 at every raw read's address (the one-window TLS
+                              // shadow slots a violator polls: no full clear of V needed)
 };
 
 template <int OP>
 __global__ void __launch_bounds__(kEvalThreads) k_bk_eval(BkView V, const uint32_t *base, const uint32_t *tot,
                                                           const unsigned long long *rec, BkOut O) {
+  if (gated(V.gate)) return;
   // dynamic: minW[8192], minR[8192] (ADD_C), then 3 x nch per-chunk counts when they fit
   extern __shared__ uint32_t s_dyn[];
   uint32_t *minW = s_dyn;
@@ -374,6 +385,7 @@ __global__ void __launch_bounds__(kEvalThreads) k_bk_eval(BkView V, const uint32
     c_raw += raw; c_war += war; c_waw += waw;
     if (raw) {
       if (O.wsrc && rec_reads(x)) O.wsrc[i] = (int32_t)jw;
+      if (O.vclr && rec_reads(x)) O.vclr[(uint32_t)b << kBShift | al] = 0ull;
       if (O.graw) atomicOr(&O.graw[i >> 5], 1u << (i & 31));
       if (O.gsrc) atomicOr(&O.gsrc[jw >> 5], 1u << (jw & 31));
       atomicAdd(&s_dist[31 - __clz(i - jw)], 1u);
@@ -447,6 +459,7 @@ constexpr uint32_t kPredCapB = (uint32_t)((kPredSmemB - kPredFixed) / 4);
 
 struct PredOut {
   int32_t *pred;                  // [n] last earlier writer of raw iteration i's read (loop-local)
+  unsigned long long *V;          // [n] per-iteration shadow slots: V[pred] = 0 for every pred
   uint32_t *pub, *now, *later;    // [nw] each, zeroed by the caller
   int64_t *hdr;                   // H_PRED_FAIL, H_PRED_SEG
   uint32_t *redo;                 // [B] bucket left to the big tier
@@ -543,6 +556,7 @@ __device__ __forceinline__ void pred_bucket(int b, const uint32_t *base, const u
     }
     if (best != 0xFFFFFFFFu) {
       O.pred[i] = (int32_t)best;
+      O.V[best] = 0ull;
       atomicOr(&O.pub[best >> 5], 1u << (best & 31));
     } else {
       atomicOr(&xflag[al >> 5], 1u << (al & 31));
@@ -577,15 +591,44 @@ __global__ void __launch_bounds__(1024, 1) k_bk_pred_big(int B, const uint32_t *
 // everything the profile accumulates into, reset in one launch: the header
 // (first raw iteration = -1), the guide words, the per-chunk counts and the
 // per-chunk address ranges (min = ~0, max = 0)
+// (with pfx: warp 0 of block 0 also runs the static check's affine sample --
+// reading B8: an index array that is not affine on its first m entries is not
+// affine -- writes the verdict to hdr[H_GATE] (1: looks affine, the profile's
+// kernels queued behind exit at once) and to mapped host words mir[0], then the
+// call's sequence number mir[1])
+struct PrefixDuty {
+  const int32_t *p[4];
+  int m;
+  long long *mir;
+  unsigned long long seq;
+};
 __global__ void __launch_bounds__(256) k_bk_prep(int64_t *hdr, uint32_t *graw, uint32_t *gsrc, int64_t nw, int64_t *cc,
-                                                 int64_t ncc, uint32_t *cr, int64_t nck) {
+                                                 int64_t ncc, uint32_t *cr, int64_t nck, PrefixDuty pfx) {
+  if (blockIdx.x == 0 && threadIdx.x < 32) {
+    bool ok = pfx.m >= 3;
+    if (ok)
+#pragma unroll
+      for (int q = 0; q < 4; q++) {
+        if (!pfx.p[q]) continue;
+        const int64_t b = __ldg(pfx.p[q]), a = (int64_t)__ldg(pfx.p[q] + 1) - b;
+        for (int k = threadIdx.x; k < pfx.m; k += 32) ok = ok && (int64_t)__ldg(pfx.p[q] + k) == b + a * k;
+      }
+    ok = __all_sync(0xffffffffu, ok);
+    if (threadIdx.x == 0) {
+      hdr[H_GATE] = ok ? 1 : 0;
+      if (pfx.mir) {
+        pfx.mir[0] = ok ? 1 : 0;
+        asm volatile("st.release.sys.global.u64 [%0], %1;" ::"l"(pfx.mir + 1), "l"(pfx.seq) : "memory");
+      }
+    }
+  }
   const int64_t nh = (int64_t)(kHeaderBytes / 8);
   int64_t m = nh;
   if (nw > m) m = nw;
   if (ncc > m) m = ncc;
   if (nck > m) m = nck;
   for (int64_t k = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; k < m; k += (int64_t)gridDim.x * blockDim.x) {
-    if (k < nh) hdr[k] = k == H_FIRST_RAW ? -1 : 0;
+    if (k < nh && k != H_GATE) hdr[k] = k == H_FIRST_RAW ? -1 : 0;
     if (k < nw) {
       if (graw) graw[k] = 0;
       if (gsrc) gsrc[k] = 0;
@@ -627,7 +670,7 @@ bool plan(const Job &j, void *ws, const Layout &lo, BkPlan &P) {
   const size_t rb = lo.bytes[R_KEYS_A] ? lo.off[R_KEYS_A] + lo.bytes[R_KEYS_A] - lo.off[R_MINW_A] : 0;
   if (!lo.bytes[R_MINW_A] || rb < 8 * (size_t)nrec) return false;
   if (lo.bytes[R_MAXRX_A] < 4 * ((size_t)T * B + 2 * (size_t)B)) return false;
-  P.v = BkView{d.r, d.w, d.n, d.ioff, (uint32_t)d.lenA, B, T, nullptr, 1};
+  P.v = BkView{d.r, d.w, d.n, d.ioff, (uint32_t)d.lenA, B, T, nullptr, 1, nullptr};
   P.rec = at<unsigned long long>(ws, lo, R_MINW_A);
   P.cnt = at<uint32_t>(ws, lo, R_MAXRX_A);
   P.tot = P.cnt + (size_t)T * B;
@@ -641,8 +684,8 @@ void run_bucket(const BkPlan &P, const DLoop &d, int64_t *hdr, BkOut O, cudaStre
   const int vec = al(d.r) && al(d.w);
   const int B = P.v.B, T = P.v.T;
   k_bk_count<OP><<<T, kBThreads, 4 * (size_t)B, st>>>(P.v, vec, P.cnt, &hdr[H_BAD]);
-  k_bk_scan_tiles<<<(B + 31) / 32, 1024, 0, st>>>(P.cnt, T, B, P.tot);
-  k_bk_scan_buckets<<<1, 1024, 0, st>>>(P.tot, B, P.base);
+  k_bk_scan_tiles<<<(B + 31) / 32, 1024, 0, st>>>(P.cnt, T, B, P.tot, P.v.gate);
+  k_bk_scan_buckets<<<1, 1024, 0, st>>>(P.tot, B, P.base, P.v.gate);
   const size_t ssm = 6 * 2 * (size_t)kTile + 4 * (3 * (size_t)B + 1);
   cudaFuncSetAttribute(k_bk_scatter<OP>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)ssm);
   k_bk_scatter<OP><<<T, kBThreads, ssm, st>>>(P.v, vec, P.cnt, P.tot, P.base, P.rec);
@@ -660,9 +703,12 @@ bool bucket_profile_ok(const Job &j, void *ws, const Layout &lo) {
 }
 
 cudaError_t launch_prof_bucket(const Job &j, void *ws, const Layout &lo, uint32_t *graw, uint32_t *gsrc,
-                               int64_t chunk, int64_t *cc, cudaStream_t st, int32_t *wsrc, uint32_t *crange) {
+                               int64_t chunk, int64_t *cc, cudaStream_t st, int32_t *wsrc, uint32_t *crange,
+                               unsigned long long *vclr, int sample_m, long long *mir, unsigned long long seq) {
   BkPlan P;
   if (!plan(j, ws, lo, P)) return cudaErrorInvalidValue;
+  PrefixDuty pfx{{j.d.r, j.d.r2, j.d.w, j.d.s}, sample_m, mir, seq};
+  if (sample_m > 0) P.v.gate = &at<int64_t>(ws, lo, R_HEADER)[H_GATE];
   static_assert(kTile == kBucketTile, "jp_host.h kBucketTile");
   int64_t nck = 0;
   if (crange && chunk > 0 && chunk % kTile == 0) {
@@ -677,17 +723,18 @@ cudaError_t launch_prof_bucket(const Job &j, void *ws, const Layout &lo, uint32_
     int64_t m = std::max<int64_t>(std::max<int64_t>((int64_t)(kHeaderBytes / 8), nw), std::max(ncc, nck));
     const int64_t need = (m + 255) / 256, cap = (int64_t)num_sms() * 4;
     k_bk_prep<<<(int)(need < cap ? need : cap), 256, 0, st>>>(hdr, graw, gsrc, nw, cc, ncc, nck ? crange : nullptr,
-                                                              nck);
+                                                              nck, pfx);
     note_launch();
   }
-  BkOut O{hdr, graw, gsrc, chunk, cc, j.d.base, j.op == JP_OP_ADD_C ? wsrc : nullptr};
+  BkOut O{hdr, graw, gsrc, chunk, cc, j.d.base, j.op == JP_OP_ADD_C ? wsrc : nullptr,
+          j.op == JP_OP_ADD_C ? vclr : nullptr};
   if (j.op == JP_OP_ADD_C) run_bucket<JP_OP_ADD_C>(P, j.d, hdr, O, st);
   else run_bucket<JP_OP_SAXPY>(P, j.d, hdr, O, st);
   return launch_check();
 }
 
 cudaError_t launch_prof_pred(const Job &j, void *ws, const Layout &lo, int32_t *pred, uint32_t *bits,
-                             cudaStream_t st) {
+                             unsigned long long *V, cudaStream_t st) {
   BkPlan P;
   if (j.op != JP_OP_ADD_C || !plan(j, ws, lo, P)) return cudaErrorInvalidValue;
   const int64_t nw = (j.d.n + 31) / 32;
@@ -699,7 +746,7 @@ cudaError_t launch_prof_pred(const Job &j, void *ws, const Layout &lo, int32_t *
   if (e == cudaSuccess)
     e = cudaFuncSetAttribute(k_bk_pred_big, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)kPredSmemB);
   if (e != cudaSuccess) return e;
-  PredOut O{pred, bits, bits + nw, bits + 2 * nw, at<int64_t>(ws, lo, R_HEADER), P.cnt};
+  PredOut O{pred, V, bits, bits + nw, bits + 2 * nw, at<int64_t>(ws, lo, R_HEADER), P.cnt};
   k_bk_pred<<<P.v.B, 512, kPredSmemS, st>>>(P.base, P.tot, P.rec, O);
   k_bk_pred_big<<<std::min(P.v.B, num_sms()), 1024, kPredSmemB, st>>>(P.v.B, P.base, P.tot, P.rec, O);
   note_launch(2);

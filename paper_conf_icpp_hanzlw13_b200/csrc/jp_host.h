@@ -79,21 +79,31 @@ cudaError_t launch_tls_flow(const Job &j, const uint32_t *graw, const uint32_t *
 // wsrc (nullable, ADD_C): the first writer of every raw iteration's read (int32 [n])
 // crange (nullable, needs chunk % 16384 == 0): per chunk the min and max address of A
 // the chunk touches (uint32 [2 * chunks]) -- the stealing scheduler's task ranges
+// vclr (nullable, ADD_C): V[a] = 0 at the address of every raw read -- every slot
+// the one-window TLS (path 8) polls or publishes, so V needs no full clear
+// sample_m > 0: the first kernel also runs the static check's affine sample on
+// the first sample_m entries of every index array (verdict to hdr[H_GATE] and to
+// the mapped host words mir[0], then seq to mir[1]); when the sample looks
+// affine every later kernel of the profile exits at once (H_GATE = 1), so the
+// host can queue the whole profile before it knows the verdict
 cudaError_t launch_prof_bucket(const Job &j, void *ws, const Layout &lo, uint32_t *graw, uint32_t *gsrc,
                                int64_t chunk, int64_t *cc, cudaStream_t st, int32_t *wsrc = nullptr,
-                               uint32_t *crange = nullptr);
+                               uint32_t *crange = nullptr, unsigned long long *vclr = nullptr, int sample_m = 0,
+                               long long *mir = nullptr, unsigned long long seq = 0);
 constexpr int64_t kBucketTile = 16384;   // (jp_bucket.cu's tile: chunk ranges need chunk % kBucketTile == 0)
 // after launch_prof_bucket on the same workspace (its records still in place),
 // ADD_C: the last earlier writer of every raw read -> pred[i] (raw i only), and
 // three bitmaps of nw = ceil(n/32) words at bits (zeroed here): publish (the
 // writer is some raw read's pred), now (last writer of an address no exposed read
 // touches), later (last writer of an address that has an exposed read).
-// hdr[H_PRED_FAIL] > 0 if the pass could not hold some bucket's writers.
+// hdr[H_PRED_FAIL] > 0 if the pass could not hold some bucket's writers.  V[pred]
+// = 0 for every pred (the only per-iteration shadow slots path 9 polls).
 cudaError_t launch_prof_pred(const Job &j, void *ws, const Layout &lo, int32_t *pred, uint32_t *bits,
-                             cudaStream_t st);
+                             unsigned long long *V, cudaStream_t st);
 // one-window on-chip TLS over a loop with WAR / WAW (path 9, reading B14): pred and
 // bits from launch_prof_pred, graw the profile's raw words, V one tagged shadow
-// slot per ITERATION (zeroed); the kernel exits at once if gate[H_PRED_FAIL] != 0.
+// slot per ITERATION (V[pred] zeroed by launch_prof_pred); the kernel exits at once
+// if gate[H_PRED_FAIL] != 0.
 // stats as launch_tls_flow's (stats[3] violations, stats[1] lost warps)
 cudaError_t launch_tls_flow_waw(const Job &j, const uint32_t *graw, const int32_t *pred, const uint32_t *bits,
                                 unsigned long long *V, int64_t *stats, const int64_t *gate, cudaStream_t st);

@@ -42,6 +42,7 @@ enum Hdr : int {
   H_BAR_COUNT = 16, H_BAR_GEN = 17, H_FV0 = 20, H_FV1 = 21, H_FV2 = 22, H_AFFINE = 24 /* 2 slots = 4 int */,
   H_PRED_FAIL = 28 /* buckets whose writers overflowed the last-writer pass (jp_bucket.cu) */,
   H_PRED_SEG = 29 /* longest writer list of one address seen by that pass */,
+  H_GATE = 30 /* nonzero: the index arrays look affine on their prefix -- the profile's kernels exit */,
   H_DIST = 64 /* 32 slots: raw reads by floor(log2(i - writer)) */, H_SLOTS = 96
 };
 constexpr size_t kHeaderBytes = 4096;

@@ -141,7 +141,8 @@ __global__ void __launch_bounds__(kFlowT, JP_FLOW_MINB) k_tls_flow(DLoop L, cons
   // gate (nullable): the profile header of this call -- launched before the host
   // has read it, the kernel runs only if the profile makes the loop a path-8 loop
   // (no bad index, war = waw = 0, 0 < raw <= raw_max, i.e. Fig. 2(b) mode B)
-  if (gate && (gate[H_BAD] != 0 || gate[H_WAR] != 0 || gate[H_WAW] != 0 || gate[H_RAW] <= 0 || gate[H_RAW] > raw_max))
+  if (gate && (gate[H_BAD] != 0 || gate[H_WAR] != 0 || gate[H_WAW] != 0 || gate[H_RAW] <= 0 || gate[H_RAW] > raw_max ||
+               gate[H_GATE] != 0))
     return;
   Flow<DT> F;
   F.L = L; F.graw = graw; F.gsrc = gsrc; F.V = V; F.wsrc = wsrc; F.lo = lo;

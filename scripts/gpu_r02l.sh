@@ -1,0 +1,5 @@
+mkdir -p gpurun_out
+timeout 1500 python -m pytest tests -m gpu -x -q > gpurun_out/pytest_gpu.log 2>&1; echo pytest=$?; tail -3 gpurun_out/pytest_gpu.log
+timeout 300 python scripts/sched3_time.py > gpurun_out/sched3.log 2>&1; echo t=$?; cat gpurun_out/sched3.log
+timeout 300 python scripts/waw_time.py > gpurun_out/waw_time.log 2>&1; echo waw=$?; cat gpurun_out/waw_time.log | tail -8
+python scripts/timeline.py config3 0.01 2>/dev/null; python scripts/timeline.py config5 2>/dev/null
