@@ -1189,7 +1189,11 @@ static jp_status run_mode(const jp_loop *L, const Job &j, int mode, const jp_pro
                           int s_clean = 0, const int64_t *dist = nullptr) {
   Layout lo = layout(L);
   if (mode == JP_MODE_DOALL) {
-    JP_CUDA(launch_doall(j, st), "doall");
+    // an indirect loop: gather phase into region 1 (the profile's scratch, free
+    // once Fig. 2(b) has its counts), then the scatters
+    uint32_t *o = ws && lo.bytes[R_MINW_A] >= 4 * (size_t)j.d.n && ws_bytes >= lo.off[R_MINW_A] + 4 * (size_t)j.d.n
+                      ? at<uint32_t>(ws, lo, R_MINW_A) : nullptr;
+    JP_CUDA(launch_doall(j, st, 0, o), "doall");
   } else if (mode == JP_MODE_PRIVATIZED) {
     if (ws_bytes < layout_end(lo, JP_WS_PRIV)) return fail(JP_ERR_WORKSPACE, "workspace too small for privatization");
     bool applied = false;
@@ -1529,7 +1533,9 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
           if (n_priv == 1) clear_keys(s2);
           JP_CUDA(launch_priv_stream(sj, ws, lo, false, s2), "priv task");
         } else {
-          JP_CUDA(launch_doall(sj, s2), "doall task");
+          // gather phase into region 1 at the task's own offset (tasks are disjoint ranges)
+          uint32_t *o = lo.bytes[R_MINW_A] >= 4 * (size_t)L->n ? at<uint32_t>(ws, lo, R_MINW_A) + tasks[t].s : nullptr;
+          JP_CUDA(launch_doall(sj, s2, 0, o), "doall task");
         }
         res->task_mode_iters[tasks[t].mode] += sj.d.n;
         cudaEvent_t e;

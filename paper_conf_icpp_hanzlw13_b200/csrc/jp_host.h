@@ -114,7 +114,10 @@ cudaError_t launch_prof_classify(const Job &j, void *ws, const Layout &lo, uint3
 // counts + the TLS guide bitmaps (region 13, valid when the loop writes no address twice) in one pass
 cudaError_t launch_prof_classify_guide(const Job &j, void *ws, const Layout &lo, cudaStream_t st,
                                        bool stamped_pairs = false);
-cudaError_t launch_doall(const Job &j, cudaStream_t st, int max_ctas = 0);
+// o (nullable, n words of scratch): an indirect loop other than PRIV_TMP runs as a
+// gather kernel (every iteration's value into o) then a scatter kernel
+// (JP_DOALL_PHASED=0 keeps the one-kernel form)
+cudaError_t launch_doall(const Job &j, cudaStream_t st, int max_ctas = 0, uint32_t *o = nullptr);
 int doall_kernel_choice();
 void set_doall_kernel_choice(int v);
 // fuse_apply: the stream kernel may also apply the keys (single-GPU PE(V));
