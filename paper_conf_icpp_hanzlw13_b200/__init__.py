@@ -26,7 +26,7 @@ __all__ = [
     "jp_profile_classify", "jp_profile_density", "jp_select_mode", "jp_run_doall", "jp_run_privatized",
     "jp_priv_stream", "jp_priv_finalize", "jp_doall_kernel", "jp_tls_guide", "jp_tls_next_window", "jp_run_tls", "jp_schedule", "jp_stage_bytes", "jp_schedule_host",
     "jp_plan_sharing", "jp_plan_stealing", "jp_merge_apply",
-    "jp_plan", "jp_plan_tasks", "jp_export_keys", "jp_keys_merge_p2p", "jp_priv_inbox_bytes", "jp_priv_stream_merge", "jp_run_priv_claim", "jp_run_doall_spill", "jp_ipc_export", "jp_ipc_import", "jp_ipc_close",
+    "jp_plan", "jp_plan_tasks", "jp_profile_plan_tasks", "jp_export_keys", "jp_keys_merge_p2p", "jp_priv_inbox_bytes", "jp_priv_stream_merge", "jp_run_priv_claim", "jp_run_doall_spill", "jp_ipc_export", "jp_ipc_import", "jp_ipc_close",
     "jp_sparse_scratch_bytes", "jp_sparse_pack", "jp_sparse_reduce_max", "jp_sparse_gather", "jp_sparse_scatter",
     "jp_last_error", "jp_version", "jp_launch_count", "jp_tls_grid_window",
 ]
@@ -378,6 +378,23 @@ def jp_plan_tasks(loop: Loop, chunk_counts, chunk_iters: int, ws, tau_high: floa
     check(lib().jp_plan_tasks(loop.ref, hc, int(chunk_iters), float(tau_high), p, nb, tk, C.byref(nt), cf,
                               _stream(stream)))
     return [(tk[3 * t], tk[3 * t + 1], tk[3 * t + 2]) for t in range(nt.value)], list(cf)
+
+
+def jp_profile_plan_tasks(loop: Loop, chunk_iters: int, ws, tau_high: float = _abi.TAU_HIGH, stream=None):
+    """The whole loop's profile (this rank's own, no exchange) with per-chunk
+    counts, then the task plan.  Returns (profile dict, chunk counts list,
+    [(start, end, mode)], conf list of 64 ints)."""
+    nck = -(-loop.n // int(chunk_iters))
+    pr = _abi.jp_profile()
+    hc = (C.c_int64 * max(3 * nck, 1))()
+    tk = (C.c_int64 * 192)()
+    nt = C.c_int32()
+    cf = (C.c_uint64 * 64)()
+    p, nb = _ws(ws)
+    check(lib().jp_profile_plan_tasks(loop.ref, int(chunk_iters), float(tau_high), p, nb, C.byref(pr), hc, tk,
+                                      C.byref(nt), cf, _stream(stream)))
+    return (_prof_dict(pr), list(hc[:3 * nck]), [(tk[3 * t], tk[3 * t + 1], tk[3 * t + 2]) for t in range(nt.value)],
+            list(cf))
 
 
 def jp_export_keys(loop: Loop, ws, stream=None):

@@ -114,6 +114,8 @@ SIGNATURES = [
     ("jp_merge_apply", _I32, [_V, _I64, _V, _V]),
     ("jp_plan", _I32, [_P(jp_loop), _P(jp_sched_cfg), _P(jp_profile), _I64, _I32, _P(_D), _P(_I64), _I64, _P(_I64)]),
     ("jp_plan_tasks", _I32, [_P(jp_loop), _P(_I64), _I64, _D, _V, _SZ, _P(_I64), _P(_I32), _P(C.c_uint64), _V]),
+    ("jp_profile_plan_tasks", _I32, [_P(jp_loop), _I64, _D, _V, _SZ, _P(jp_profile), _P(_I64), _P(_I64), _P(_I32),
+                                     _P(C.c_uint64), _V]),
     ("jp_export_keys", _I32, [_P(jp_loop), _V, _SZ, _V]),
     ("jp_run_priv_claim", _I32, [_P(jp_loop), _V, _P(_I64), _I32, _I32, _V, _V, _V, _SZ, _I32, _V]),
     ("jp_keys_merge_p2p", _I32, [_P(_V), _I32, _V, _I64, _V, _I64, _V, _V, _V]),

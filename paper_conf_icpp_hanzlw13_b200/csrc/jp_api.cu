@@ -1289,6 +1289,84 @@ static std::vector<Task> chunk_tasks(const int64_t *hc, int64_t n, int64_t chunk
 // ([4][kMaxTasks]: minA, maxA, minT, maxT) when it ran, else left empty
 // chunk_rg (nullable): per chunk the min / max address of A it touches (the bucket
 // profile's), from which the task ranges follow without the k_task_ranges pass
+// Small device-to-host reads of the schedulers through mapped pinned memory:
+// one kernel copies up to three device ranges (8-byte words) into the mapped
+// buffer and then publishes the call's sequence number; the host polls it.
+namespace {
+struct MappedPack {
+  char *host = nullptr, *dev = nullptr;
+  size_t bytes = 0;
+  unsigned long long *flag_host = nullptr, *flag_dev = nullptr;
+  unsigned long long seq = 0;
+};
+}  // namespace
+__global__ void __launch_bounds__(256) k_pack_host(const unsigned long long *a, size_t na, const unsigned long long *b,
+                                                   size_t nb, const unsigned long long *c, size_t nc,
+                                                   unsigned long long *dst, unsigned long long *flag,
+                                                   unsigned long long seq) {
+  for (size_t k = threadIdx.x; k < na + nb + nc; k += blockDim.x)
+    dst[k] = k < na ? a[k] : k < na + nb ? b[k - na] : c[k - na - nb];
+  __threadfence_system();
+  JP_CTA_SYNC();
+  if (threadIdx.x == 0) asm volatile("st.release.sys.global.u64 [%0], %1;" ::"l"(flag), "l"(seq) : "memory");
+}
+static MappedPack &mapped_pack(size_t need) {
+  thread_local MappedPack m;
+  if (need > m.bytes && !getenv("JP_NO_MAPPED_PACK")) {
+    if (m.host) cudaFreeHost(m.host);
+    m = MappedPack{};
+    void *p = nullptr, *d = nullptr;
+    const size_t bytes = ((need + 4095) & ~(size_t)4095) + 64;
+    if (cudaHostAlloc(&p, bytes, cudaHostAllocMapped | cudaHostAllocPortable) == cudaSuccess) {
+      if (cudaHostGetDevicePointer(&d, p, 0) == cudaSuccess) {
+        m.host = static_cast<char *>(p);
+        m.dev = static_cast<char *>(d);
+        m.bytes = bytes - 64;
+        m.flag_host = reinterpret_cast<unsigned long long *>(m.host + m.bytes);
+        m.flag_dev = reinterpret_cast<unsigned long long *>(m.dev + m.bytes);
+        *m.flag_host = 0;
+      } else {
+        cudaFreeHost(p);
+      }
+    }
+    cudaGetLastError();
+  }
+  return m;
+}
+static cudaError_t launch_pack_host(const void *a, size_t ba, const void *b, size_t bb, const void *c, size_t bc,
+                                    char *dst, unsigned long long seq, cudaStream_t st) {
+  MappedPack &m = mapped_pack(ba + bb + bc);
+  k_pack_host<<<1, 256, 0, st>>>(static_cast<const unsigned long long *>(a), ba / 8,
+                                 static_cast<const unsigned long long *>(b), bb / 8,
+                                 static_cast<const unsigned long long *>(c), bc / 8,
+                                 reinterpret_cast<unsigned long long *>(dst), m.flag_dev, seq);
+  note_launch();
+  return launch_check();
+}
+static jp_status mapped_pack_wait(MappedPack &m, unsigned long long seq, cudaStream_t st, const char *what) {
+  volatile unsigned long long *flag = m.flag_host;
+  for (unsigned spins = 0; *flag != seq; spins++) {
+    if ((spins & 1023) == 1023) {
+      const cudaError_t q = cudaStreamQuery(st);
+      if (q != cudaSuccess && q != cudaErrorNotReady) return cuda_fail(q, what);
+      if (q == cudaSuccess && *flag != seq) return fail(JP_ERR_CUDA, "%s: the pack kernel did not publish", what);
+    }
+  }
+  return JP_OK;
+}
+
+#include <chrono>
+// host-side phase trace of the schedulers (JP_HOST_TRACE=1: microseconds since the previous mark, stderr)
+static void htrace(const char *what) {
+  static const bool on = getenv("JP_HOST_TRACE") != nullptr;
+  if (!on) return;
+  thread_local auto prev = std::chrono::steady_clock::now();
+  const auto now = std::chrono::steady_clock::now();
+  fprintf(stderr, "[jp host] %-16s +%.1f us\n", what, std::chrono::duration<double, std::micro>(now - prev).count());
+  prev = now;
+}
+#define HTRACE(w) htrace(w)
+
 static jp_status task_conflicts(const Job &j, const jp_loop *L, void *ws, const Layout &lo,
                                 const std::vector<Task> &tasks, int64_t chunk, std::vector<unsigned long long> &conf,
                                 cudaStream_t st, std::vector<uint32_t> *ranges_out = nullptr,
@@ -1347,8 +1425,78 @@ static jp_status task_conflicts(const Job &j, const jp_loop *L, void *ws, const 
   return JP_OK;
 }
 
+// Step 1 of the stealing schedulers: the profile of the whole loop with per-chunk
+// (raw, war, waw) counts (global stamps, reading A19) -- by address buckets when
+// the loop allows it, with the per-chunk address ranges of A (the task PDG's
+// prefilter) -- read back to the host: hc [3 nck], hcr [2 nck] (empty without
+// ranges), h = header words 0..7.  gbits (nullable): the TLS guide words are
+// written too; flow: keep the writer of every raw read (wsrc, region 7) and clear
+// the shadow slots path 8 polls (vclr) for one-window TLS tasks.
+static jp_status chunk_profile(const jp_loop *L, const Job &j, void *ws, const Layout &lo, int64_t chunk,
+                               uint32_t *gbits, bool pairs, bool flow, cudaStream_t st, std::vector<int64_t> &hc,
+                               std::vector<uint32_t> &hcr, std::vector<int64_t> &h, int32_t **wsrc_out,
+                               uint32_t **crange_out, unsigned long long **vclr_out, bool *bucket_out) {
+  SchedLayout sl = sched_layout(L);
+  char *sch = static_cast<char *>(ws) + lo.off[R_SCHED];
+  const int64_t nck = (L->n + chunk - 1) / chunk;
+  int64_t *cc = reinterpret_cast<int64_t *>(sch + sl.counts);
+  int32_t *wsrc = nullptr;
+  uint32_t *crange = nullptr;
+  unsigned long long *vclr = nullptr;
+  const bool bucket = bucket_profile_ok(j, ws, lo);
+  if (bucket) {   // large A: the profile by address buckets (jp_bucket.cu)
+    if (flow && gbits && j.op == JP_OP_ADD_C && lo.bytes[R_TLS_S_A] >= 4 * (size_t)L->n && !getenv("JP_TLS_NO_FLOW"))
+      wsrc = at<int32_t>(ws, lo, R_TLS_S_A);
+    if (chunk % kBucketTile == 0 && !getenv("JP_TASK_MASKS_ALWAYS"))
+      crange = reinterpret_cast<uint32_t *>(sch + sl.crange);
+    // the shadow slots a one-window TLS task polls (V at every raw read's
+    // address) are cleared by the profile itself
+    vclr = wsrc ? at<unsigned long long>(ws, lo, R_TLS_C_A) : nullptr;
+    JP_CUDA(launch_prof_bucket(j, ws, lo, gbits, gbits ? gbits + (L->n + 31) / 32 : nullptr, chunk, cc, st, wsrc,
+                               crange, vclr),
+            "profile (buckets)");
+  } else {
+    JP_CUDA(launch_prof_stamp(j, ws, lo, st, pairs), "profile stamp");
+    JP_CUDA(launch_prof_classify(j, ws, lo, gbits, chunk, cc, st, gbits ? gbits + (L->n + 31) / 32 : nullptr, pairs),
+            "profile classify");
+  }
+  hc.assign(3 * nck, 0);
+  h.assign(8, 0);
+  hcr.clear();
+  {
+    // chunk counts, chunk address ranges and the header: one kernel stores them
+    // into mapped pinned memory and then a sequence word, which the host polls
+    // (three DMA copies and a stream sync cost ~20 us more); the copies stay as
+    // the fallback when mapped memory is unavailable
+    const size_t bc = 24 * (size_t)nck, br = crange ? 8 * (size_t)nck : 0, bh = 64;
+    if (crange) hcr.resize(2 * nck);
+    HTRACE("profile queued");
+    MappedPack &mp = mapped_pack(bc + br + bh);
+    if (mp.host) {
+      const unsigned long long seq = ++mp.seq;
+      JP_CUDA(launch_pack_host(cc, bc, crange, br, at<int64_t>(ws, lo, R_HEADER), bh, mp.dev, seq, st), "profile D2H");
+      JP_TRY(mapped_pack_wait(mp, seq, st, "profile D2H"));
+      HTRACE("pack seen");
+      memcpy(hc.data(), mp.host, bc);
+      if (crange) memcpy(hcr.data(), mp.host + bc, br);
+      memcpy(h.data(), mp.host + bc + br, bh);
+    } else {
+      JP_CUDA(cudaMemcpyAsync(hc.data(), cc, bc, cudaMemcpyDeviceToHost, st), "chunk D2H");
+      if (crange) JP_CUDA(cudaMemcpyAsync(hcr.data(), crange, br, cudaMemcpyDeviceToHost, st), "chunk ranges D2H");
+      JP_CUDA(cudaMemcpyAsync(h.data(), at<int64_t>(ws, lo, R_HEADER), bh, cudaMemcpyDeviceToHost, st), "profile D2H");
+      JP_CUDA(cudaStreamSynchronize(st), "profile sync");
+    }
+  }
+  if (wsrc_out) *wsrc_out = wsrc;
+  if (crange_out) *crange_out = crange;
+  if (vclr_out) *vclr_out = vclr;
+  if (bucket_out) *bucket_out = bucket;
+  return JP_OK;
+}
+
 static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sched_cfg &c, void *ws, size_t ws_bytes,
                                    jp_sched_result *res, cudaStream_t st) {
+  HTRACE("start");
   const int64_t chunk = c.chunk_iters;
   if (chunk < kSchedMinChunk || chunk % 32) return fail(JP_ERR_ARG, "stealing needs chunk_iters >= 1024, multiple of 32");
   Layout lo;
@@ -1374,55 +1522,15 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
   int32_t *wsrc = nullptr;
   uint32_t *crange = nullptr;   // per-chunk address ranges from the bucket profile (task PDG prefilter)
   unsigned long long *vclr = nullptr;   // the shadow values, cleared where path 8 polls them by the profile
-  if (bucket_profile_ok(j, ws, lo)) {   // large A: the profile by address buckets (jp_bucket.cu)
-    s_fresh = false;                    // (region 7 is not filled: the TLS task resets it)
-    if (gbits && j.op == JP_OP_ADD_C && lo.bytes[R_TLS_S_A] >= 4 * (size_t)L->n && !getenv("JP_TLS_NO_FLOW"))
-      wsrc = at<int32_t>(ws, lo, R_TLS_S_A);
-    if (chunk % kBucketTile == 0 && !getenv("JP_TASK_MASKS_ALWAYS"))
-      crange = reinterpret_cast<uint32_t *>(sch + sl.crange);
-    // the shadow slots a one-window TLS task polls (V at every raw read's
-    // address) are cleared by the profile itself
-    vclr = wsrc ? at<unsigned long long>(ws, lo, R_TLS_C_A) : nullptr;
-    JP_CUDA(launch_prof_bucket(j, ws, lo, gbits, gbits ? gbits + (L->n + 31) / 32 : nullptr, chunk, cc, st, wsrc,
-                               crange, vclr),
-            "profile (buckets)");
-  } else {
-    JP_CUDA(launch_prof_stamp(j, ws, lo, st, pairs), "profile stamp");
-    JP_CUDA(launch_prof_classify(j, ws, lo, gbits, chunk, cc, st, gbits ? gbits + (L->n + 31) / 32 : nullptr, pairs),
-            "profile classify");
-  }
   std::vector<int64_t> hc(3 * nck), h(8);
   std::vector<uint32_t> hcr;
-  {
-    // chunk counts, chunk address ranges and the header through one pinned
-    // staging buffer (pageable copies each stall the host)
-    thread_local char *pin = nullptr;
-    thread_local size_t pin_bytes = 0;
-    const size_t need = 24 * (size_t)nck + (crange ? 8 * (size_t)nck : 0) + 64;
-    if (need > pin_bytes) {
-      if (pin) cudaFreeHost(pin);
-      pin = nullptr;
-      pin_bytes = 0;
-      if (cudaMallocHost(reinterpret_cast<void **>(&pin), need) == cudaSuccess) pin_bytes = need;
-      else cudaGetLastError();
-    }
-    char *dst_c = pin ? pin : reinterpret_cast<char *>(hc.data());
-    if (crange) hcr.resize(2 * nck);
-    char *dst_r = pin ? pin + 24 * nck : reinterpret_cast<char *>(hcr.data());
-    char *dst_h = pin ? pin + 24 * nck + (crange ? 8 * nck : 0) : reinterpret_cast<char *>(h.data());
-    JP_CUDA(cudaMemcpyAsync(dst_c, cc, 24 * nck, cudaMemcpyDeviceToHost, st), "chunk D2H");
-    if (crange) JP_CUDA(cudaMemcpyAsync(dst_r, crange, 8 * nck, cudaMemcpyDeviceToHost, st), "chunk ranges D2H");
-    JP_CUDA(cudaMemcpyAsync(dst_h, at<int64_t>(ws, lo, R_HEADER), 64, cudaMemcpyDeviceToHost, st), "profile D2H");
-    JP_CUDA(cudaStreamSynchronize(st), "profile sync");
-    if (pin) {
-      memcpy(hc.data(), dst_c, 24 * nck);
-      if (crange) memcpy(hcr.data(), dst_r, 8 * nck);
-      memcpy(h.data(), dst_h, 64);
-    }
-  }
+  bool bucket = false;
+  JP_TRY(chunk_profile(L, j, ws, lo, chunk, gbits, pairs, true, st, hc, hcr, h, &wsrc, &crange, &vclr, &bucket));
+  if (bucket) s_fresh = false;   // (region 7 is not filled: the TLS task resets it)
   if (h[H_BAD]) return fail(JP_ERR_INDEX, "%lld index entries are outside their arrays", (long long)h[H_BAD]);
   fill_profile(&res->prof, L->n, h.data());
   res->profiled = 1;
+  HTRACE("copied");
   // 2. chunk modes -> tasks (maximal same-mode runs)
   std::vector<Task> tasks = chunk_tasks(hc.data(), L->n, chunk, c.tau_high);
   const int nt = (int)tasks.size();
@@ -1440,6 +1548,7 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
     nlev = std::max(nlev, level[u] + 1);
   }
   res->n_batches = nlev;
+  HTRACE("planned");
   // 4. run batch by batch; tasks of one batch are pairwise conflict-free and run
   //    concurrently (TLS on one SM, partitioned modes on the rest)
   int64_t *tstats = reinterpret_cast<int64_t *>(sch + sl.tstats);
@@ -1452,6 +1561,7 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
   // the side-stream clear (done long before: it overlapped the profile) is
   // joined before any task runs
   bool v_zeroed = vclr != nullptr;
+  const bool flow_side = !getenv("JP_FLOW_TASK_AFTER");   // path-8 tasks beside the partitioned ones
   cudaEvent_t ev0;
   JP_CUDA(cudaEventCreateWithFlags(&ev0, cudaEventDisableTiming), "event");
   std::vector<cudaEvent_t> evs;
@@ -1489,6 +1599,7 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
     };
     if (n_priv > 1) clear_keys(st);
     cudaEventRecord(ev0, st);
+    HTRACE("ev0");
     int sidx = 0;
     std::vector<cudaEvent_t> joins;
     // TLS tasks first so that their single CTA is resident before the wide grids
@@ -1513,7 +1624,27 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
           tprof.raw_iters = hc.empty() ? -1 : 0;
           for (int64_t k = tasks[t].s / chunk; k * chunk < tasks[t].e; k++) { tprof.raw_iters += hc[3 * k]; tprof.waw_iters += hc[3 * k + 2]; }
           const bool onchip = c.tls_recovery == 2 || (c.tls_recovery == 0 && c.tls_path == 0 && tprof.waw_iters == 0);
-          if (onchip) {
+          int64_t twar = 0;
+          for (int64_t k = tasks[t].s / chunk; k * chunk < tasks[t].e; k++) twar += hc[3 * k + 1];
+          if (onchip && flow_side && wsrc && guided_ok && twar == 0 && c.tls_window == 0) {
+            // write-once, WAR-free ADD_C task as one window (path 8) BESIDE the
+            // batch's partitioned tasks: one CTA per SM, so the random-access-bound
+            // sweep overlaps their streams (its violators only wait on earlier
+            // iterations of the task; the partitioned tasks never wait on it)
+            const uint32_t *gb = at<uint32_t>(ws, lo, R_GUIDE);
+            const int64_t nw = (L->n + 31) / 32;
+            auto *V = at<unsigned long long>(ws, lo, R_TLS_C_A);
+            if (!v_zeroed) cudaMemsetAsync(V, 0, lo.bytes[R_TLS_C_A], s2);
+            JP_CUDA(launch_tls_flow(sj, gb + tasks[t].s / 32, gb + nw + tasks[t].s / 32, V, tstats + 4 * t, s2,
+                                    wsrc + tasks[t].s, tasks[t].s, nullptr, 0, true, num_sms()),
+                    "tls task (one window)");
+            flow_tasks.push_back(t);
+            res->tls_w_max = sj.d.n;
+            res->tls_path = 8;
+            res->tls_recovery = JP_TLS_ONCHIP;
+            res->tls_cluster = num_sms();
+            res->tls_guided = 1;
+          } else if (onchip) {
             // on-chip recovery (reading B7) uses every SM: it runs after the
             // batch's partitioned tasks (below), on the caller's stream
             grid_tls.push_back(t);
@@ -1543,8 +1674,10 @@ static jp_status schedule_stealing(const jp_loop *L, const Job &j, const jp_sche
         cudaEventRecord(e, s2);
         joins.push_back(e);
         evs.push_back(e);
+        HTRACE("task launched");
       }
     }
+    HTRACE("tasks launched");
     for (auto e : joins) cudaStreamWaitEvent(st, e, 0);
     for (int t : grid_tls) {
       if (level[t] != lv) continue;
@@ -1684,6 +1817,38 @@ jp_status jp_plan_tasks(const jp_loop *L, const int64_t *chunk_counts, int64_t c
   std::vector<Task> tk = chunk_tasks(chunk_counts, L->n, chunk_iters, tau_high > 0.0 ? tau_high : kTauHigh);
   std::vector<unsigned long long> cf;
   JP_TRY(task_conflicts(make_job(L), L, ws, lo, tk, chunk_iters, cf, (cudaStream_t)st));
+  *n_tasks = (int32_t)tk.size();
+  for (size_t t = 0; t < tk.size(); t++) {
+    tasks[3 * t] = tk[t].s;
+    tasks[3 * t + 1] = tk[t].e;
+    tasks[3 * t + 2] = tk[t].mode;
+  }
+  for (int t = 0; t < kMaxTasks; t++) conf[t] = cf[t];
+  return JP_OK;
+}
+
+jp_status jp_profile_plan_tasks(const jp_loop *L, int64_t chunk_iters, double tau_high, void *ws, size_t ws_bytes,
+                                jp_profile *prof, int64_t *chunk_counts, int64_t *tasks, int32_t *n_tasks,
+                                uint64_t *conf, jp_stream_t stp) {
+  JP_TRY(check_loop(L));
+  if (!prof || !chunk_counts || !tasks || !n_tasks || !conf) return fail(JP_ERR_ARG, "NULL output");
+  if (chunk_iters < kSchedMinChunk || chunk_iters % 32)
+    return fail(JP_ERR_ARG, "chunk_iters must be >= 1024 and a multiple of 32");
+  JP_TRY(need_device());
+  Layout lo;
+  JP_TRY(check_ws(L, ws, ws_bytes, JP_WS_ALL, lo));
+  cudaStream_t st = (cudaStream_t)stp;
+  const Job j = make_job(L);
+  std::vector<int64_t> hc, h;
+  std::vector<uint32_t> hcr;
+  JP_TRY(chunk_profile(L, j, ws, lo, chunk_iters, nullptr, stamp_pairs_ok(j, ws, lo), false, st, hc, hcr, h, nullptr,
+                       nullptr, nullptr, nullptr));
+  if (h[H_BAD]) return fail(JP_ERR_INDEX, "%lld index entries are outside their arrays", (long long)h[H_BAD]);
+  fill_profile(prof, L->n, h.data());
+  memcpy(chunk_counts, hc.data(), hc.size() * sizeof(int64_t));
+  std::vector<Task> tk = chunk_tasks(hc.data(), L->n, chunk_iters, tau_high > 0.0 ? tau_high : kTauHigh);
+  std::vector<unsigned long long> cf;
+  JP_TRY(task_conflicts(j, L, ws, lo, tk, chunk_iters, cf, st, nullptr, hcr.empty() ? nullptr : &hcr));
   *n_tasks = (int32_t)tk.size();
   for (size_t t = 0; t < tk.size(); t++) {
     tasks[3 * t] = tk[t].s;

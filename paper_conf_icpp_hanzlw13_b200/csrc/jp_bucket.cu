@@ -687,11 +687,11 @@ void run_bucket(const BkPlan &P, const DLoop &d, int64_t *hdr, BkOut O, cudaStre
   k_bk_scan_tiles<<<(B + 31) / 32, 1024, 0, st>>>(P.cnt, T, B, P.tot, P.v.gate);
   k_bk_scan_buckets<<<1, 1024, 0, st>>>(P.tot, B, P.base, P.v.gate);
   const size_t ssm = 6 * 2 * (size_t)kTile + 4 * (3 * (size_t)B + 1);
-  cudaFuncSetAttribute(k_bk_scatter<OP>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)ssm);
+  set_smem_once((const void *)k_bk_scatter<OP>, (int)ssm);
   k_bk_scatter<OP><<<T, kBThreads, ssm, st>>>(P.v, vec, P.cnt, P.tot, P.base, P.rec);
   const int nch = O.cc ? (int)((d.n + O.chunk - 1) / O.chunk) : 0;
   const size_t sm = 4 * (size_t)kBSpan * (OP == JP_OP_ADD_C ? 2 : 1) + (O.cc && nch <= kSmemChunks ? 12 * (size_t)nch : 0);
-  cudaFuncSetAttribute(k_bk_eval<OP>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sm);
+  set_smem_once((const void *)k_bk_eval<OP>, (int)sm);
   k_bk_eval<OP><<<B, kEvalThreads, sm, st>>>(P.v, P.base, P.tot, P.rec, O);
   note_launch(5);
 }
@@ -742,9 +742,9 @@ cudaError_t launch_prof_pred(const Job &j, void *ws, const Layout &lo, int32_t *
   // redo flags in the per-tile offsets (P.cnt: the scatter was their last reader)
   if (e == cudaSuccess) e = cudaMemsetAsync(P.cnt, 0, 4 * (size_t)P.v.B, st);
   if (e == cudaSuccess)
-    e = cudaFuncSetAttribute(k_bk_pred, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)kPredSmemS);
+    e = set_smem_once((const void *)k_bk_pred, (int)kPredSmemS);
   if (e == cudaSuccess)
-    e = cudaFuncSetAttribute(k_bk_pred_big, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)kPredSmemB);
+    e = set_smem_once((const void *)k_bk_pred_big, (int)kPredSmemB);
   if (e != cudaSuccess) return e;
   PredOut O{pred, V, bits, bits + nw, bits + 2 * nw, at<int64_t>(ws, lo, R_HEADER), P.cnt};
   k_bk_pred<<<P.v.B, 512, kPredSmemS, st>>>(P.base, P.tot, P.rec, O);

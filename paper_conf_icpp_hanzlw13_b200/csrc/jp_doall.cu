@@ -12,9 +12,31 @@
 #include <atomic>
 #include <cstdlib>
 #include <cstring>
+#include <mutex>
+#include <vector>
 #include "jp_host.h"
 
 namespace jp {
+
+cudaError_t set_smem_once(const void *fn, int bytes) {
+  struct Ent { const void *fn; int dev, bytes; };
+  static std::mutex mu;
+  static std::vector<Ent> done;
+  int dev = 0;
+  cudaGetDevice(&dev);
+  {
+    std::lock_guard<std::mutex> g(mu);
+    for (const Ent &e : done)
+      if (e.fn == fn && e.dev == dev && e.bytes >= bytes) return cudaSuccess;
+  }
+  const cudaError_t e = cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, bytes);
+  if (e == cudaSuccess) {
+    std::lock_guard<std::mutex> g(mu);
+    done.push_back({fn, dev, bytes});
+  }
+  return e;
+}
+
 
 template <int OP, int DT>
 __device__ __forceinline__ void vec_body(const uint4 &x, uint4 &a, uint4 &t, uint32_t c0, uint32_t c1) {
@@ -319,7 +341,7 @@ static void run_doall(const DLoop &d, cudaStream_t st, int max_ctas) {
   if (doall_kernel_choice() == 1 && affine && aligned16(d.A) && (!d.X || aligned16(d.X)) && (!d.T || aligned16(d.T))) {
     const int64_t ntiles = d.n / kTmaTile;
     const size_t smem = (size_t)kTmaStages * 2 * kTmaTile * 4;
-    cudaFuncSetAttribute(k_doall_affine_tma<OP, DT>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+    set_smem_once((const void *)k_doall_affine_tma<OP, DT>, (int)smem);
     int64_t cap = sms;
     if (max_ctas > 0 && cap > max_ctas) cap = max_ctas;
     const int grid = (int)(ntiles < 1 ? 1 : ntiles < cap ? ntiles : cap);

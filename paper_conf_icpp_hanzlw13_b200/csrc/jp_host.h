@@ -19,6 +19,11 @@ struct Layout {
   size_t total;
 };
 
+// cudaFuncSetAttribute(fn, MaxDynamicSharedMemorySize, bytes) once per (kernel,
+// device) and size: the attribute call costs about a microsecond of host time on
+// every launch otherwise (the launch-bound front of jp_schedule)
+cudaError_t set_smem_once(const void *fn, int bytes);
+
 // Fixed-offset layout of a workspace for loop L (offsets do not depend on uses).
 Layout layout(const jp_loop *L);
 // End of the furthest region the JP_WS_* uses touch.
@@ -75,7 +80,8 @@ bool bucket_profile_ok(const Job &j, void *ws, const Layout &lo);
 // H_WAW = 0 and 0 < H_RAW <= raw_max
 cudaError_t launch_tls_flow(const Job &j, const uint32_t *graw, const uint32_t *gsrc, unsigned long long *V,
                             int64_t *stats, cudaStream_t st, const int32_t *wsrc = nullptr, int64_t lo = 0,
-                            const int64_t *gate = nullptr, int64_t raw_max = 0, bool zero_stats = true);
+                            const int64_t *gate = nullptr, int64_t raw_max = 0, bool zero_stats = true,
+                            int max_ctas = 0);
 // wsrc (nullable, ADD_C): the first writer of every raw iteration's read (int32 [n])
 // crange (nullable, needs chunk % 16384 == 0): per chunk the min and max address of A
 // the chunk touches (uint32 [2 * chunks]) -- the stealing scheduler's task ranges

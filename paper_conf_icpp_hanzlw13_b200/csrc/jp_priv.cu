@@ -528,7 +528,7 @@ static void run_priv(const DLoop &d0, unsigned long long *kA, unsigned long long
       if (doall_kernel_choice() == 1) {   // bulk-copy staged (the DOALL kernel choice covers both streams)
         const int64_t ntiles = d.n / kPrivTile;
         const size_t smem = (size_t)kPrivStages * 2 * kPrivTile * 4 + (size_t)d.lenT * 4;
-        cudaFuncSetAttribute(k_priv_tmp_tma<DT>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+        set_smem_once((const void *)k_priv_tmp_tma<DT>, (int)smem);
         int g = num_sms();
         if (max_ctas > 0 && g > max_ctas) g = max_ctas;
         if (ntiles < g) g = (int)(ntiles < 1 ? 1 : ntiles);
@@ -562,7 +562,7 @@ static void run_priv(const DLoop &d0, unsigned long long *kA, unsigned long long
           const unsigned long long bit = 1ull << (dev & 63);
           if (!(attr.load() & bit)) {
             const size_t smax = (size_t)kPh * kPh2Tile * 4 + (size_t)kSmemSlots * 4;
-            if (cudaFuncSetAttribute(k_priv_tmp_2ph<DT>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smax) ==
+            if (set_smem_once((const void *)k_priv_tmp_2ph<DT>, (int)smax) ==
                 cudaSuccess)
               attr.fetch_or(bit);
           }
@@ -623,7 +623,7 @@ cudaError_t launch_priv_stream_merge(const Job &j, unsigned long long *kT, unsig
   const size_t smem = (size_t)kPrivStages * 2 * kPrivTile * 4 + (size_t)d.lenT * 4;
   cudaError_t e;
   auto go = [&](auto kern) {
-    cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+    set_smem_once((const void *)kern, (int)smem);
     int g = num_sms();
     if (ntiles < g) g = (int)(ntiles < 1 ? 1 : ntiles);
     MergeP2P M{};
@@ -905,7 +905,7 @@ cudaError_t launch_keys_merge_p2p(const unsigned long long *const *peers, int wo
   PeerKeys P;
   for (int k = 0; k < kMaxPeers; k++) P.k[k] = k < world ? peers[k] : nullptr;
   const size_t smem = 8 * (size_t)(len > 0 ? len : 1);
-  if (smem > 48 * 1024) cudaFuncSetAttribute(k_keys_merge_p2p, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+  if (smem > 48 * 1024) set_smem_once((const void *)k_keys_merge_p2p, (int)smem);
   k_keys_merge_p2p<<<1, 1024, smem, st>>>(P, world, mine, len, bar, epoch, arr, err);
   note_launch();
   return launch_check();

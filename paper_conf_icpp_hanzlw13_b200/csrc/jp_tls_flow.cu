@@ -175,11 +175,12 @@ __global__ void __launch_bounds__(kFlowT, JP_FLOW_MINB) k_tls_flow(DLoop L, cons
 template <int DT>
 static cudaError_t run_flow(const Job &j, const uint32_t *graw, const uint32_t *gsrc, unsigned long long *V,
                             int64_t *stats, cudaStream_t st, const int32_t *wsrc, uint32_t lo, const int64_t *gate,
-                            int64_t raw_max) {
-  int maxb = 0;
-  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&maxb, (const void *)k_tls_flow<DT>, kFlowT, 0);
+                            int64_t raw_max, int max_ctas) {
+  static int maxb = 0;   // (one device model per process: B200)
+  if (maxb < 1) cudaOccupancyMaxActiveBlocksPerMultiprocessor(&maxb, (const void *)k_tls_flow<DT>, kFlowT, 0);
   if (maxb < 1) return cudaErrorInvalidConfiguration;
   int grid = num_sms() * maxb;
+  if (max_ctas > 0 && grid > max_ctas) grid = max_ctas;
   const int64_t need = (j.d.n + kFlowT - 1) / kFlowT;
   if (need < grid) grid = (int)(need < 1 ? 1 : need);
   DLoop d = j.d;
@@ -358,12 +359,12 @@ cudaError_t launch_tls_flow_waw(const Job &j, const uint32_t *graw, const int32_
 // tagged 1 << 32 for an address the loop writes (zeroed).
 cudaError_t launch_tls_flow(const Job &j, const uint32_t *graw, const uint32_t *gsrc, unsigned long long *V,
                             int64_t *stats, cudaStream_t st, const int32_t *wsrc, int64_t lo, const int64_t *gate,
-                            int64_t raw_max, bool zero_stats) {
+                            int64_t raw_max, bool zero_stats, int max_ctas) {
   if (zero_stats) cudaMemsetAsync(stats, 0, 4 * sizeof(int64_t), st);
   if (j.d.n == 0) return launch_check();
   if (j.op != JP_OP_ADD_C) return cudaErrorInvalidValue;
-  cudaError_t e = j.dt == JP_F32 ? run_flow<JP_F32>(j, graw, gsrc, V, stats, st, wsrc, (uint32_t)lo, gate, raw_max)
-                                 : run_flow<JP_I32>(j, graw, gsrc, V, stats, st, wsrc, (uint32_t)lo, gate, raw_max);
+  cudaError_t e = j.dt == JP_F32 ? run_flow<JP_F32>(j, graw, gsrc, V, stats, st, wsrc, (uint32_t)lo, gate, raw_max, max_ctas)
+                                 : run_flow<JP_I32>(j, graw, gsrc, V, stats, st, wsrc, (uint32_t)lo, gate, raw_max, max_ctas);
   if (e != cudaSuccess) return e;
   return launch_check();
 }

@@ -393,15 +393,19 @@ def _levels(conf, nt):
 
 def schedule_stealing(full, ws, group=None, chunk_iters: int = 65536, tau_high: float = _abi.TAU_HIGH, speed=None,
                       speed_tls: float = 1.0, exchange: str = "dense", engine=None, timings: bool = False,
-                      dynamic: bool = False, force_ranks: bool = False) -> dict:
+                      dynamic: bool = False, force_ranks: bool = False, profile: str = "replicated") -> dict:
     """Task stealing of one loop across the ranks (Alg. 1; SURVEY
     Sec.8(e) "Mixed").  Every rank holds full replicas (``full``, workspace
     ``ws`` of the whole loop):
 
-      1. partitioned profile with per-chunk counts: rank k stamps its
-         chunk-aligned range, C1, classifies its chunks, then C3 (SUM) of the
-         whole chunk-count array and of the totals;
-      2. jp_plan_tasks on every rank (identical): tasks = maximal same-mode chunk
+      1. profile with per-chunk counts.  ``profile="replicated"`` (default):
+         every rank profiles its full replica itself (jp_profile_plan_tasks:
+         the address-bucket profile when the loop allows it, which also records
+         per-chunk address ranges for the PDG) -- no exchange, and cheaper than
+         exchanging len(A)-sized stamp tables once A is large; ``"partitioned"``:
+         rank k stamps its chunk-aligned range, C1, classifies its chunks, then
+         C3 (SUM) of the whole chunk-count array and of the totals;
+      2. the plan on every rank (identical): tasks = maximal same-mode chunk
          runs, PDG from the per-address task masks (reading B2), batches;
       3. jp_plan_stealing: chunk owners by Alg. 1 (TLS tasks pinned to rank 0,
          tails stolen by idle ranks, reading A18);
@@ -453,24 +457,31 @@ def schedule_stealing(full, ws, group=None, chunk_iters: int = 65536, tau_high: 
             ev.record()
             marks.append((name, ev))
     mark("start")
-    c0, c1 = rank * nck // world, (rank + 1) * nck // world
-    b, e = min(c0 * chunk_iters, n), min(c1 * chunk_iters, n)
-    loop = full.range(b, e)
-    dev = ws.device
-    cc_loc = torch.zeros(max(3 * (c1 - c0), 3), dtype=torch.int64, device=dev)
-    prof = profile_partitioned(loop, ws, group, jp, exchange, chunk_iters, cc_loc)
-    cc = torch.zeros(3 * nck, dtype=torch.int64, device=dev)
-    cc[3 * c0:3 * c1] = cc_loc[:3 * (c1 - c0)]
-    if world > 1:
-        dist.all_reduce(cc, group=group)
-    mark("profile")
-    tasks, conf = jp.jp_plan_tasks(full, cc.cpu(), chunk_iters, ws, tau_high)
+    if profile == "replicated" and hasattr(jp, "jp_profile_plan_tasks"):
+        # every rank profiles its full replica itself (the address-bucket profile
+        # with per-chunk counts and address ranges): no C1 / C3 exchange, the same
+        # counts, tasks and PDG on every rank
+        prof, ccl, tasks, conf = jp.jp_profile_plan_tasks(full, chunk_iters, ws, tau_high)
+        mark("profile")
+    else:
+        c0, c1 = rank * nck // world, (rank + 1) * nck // world
+        b, e = min(c0 * chunk_iters, n), min(c1 * chunk_iters, n)
+        loop = full.range(b, e)
+        dev = ws.device
+        cc_loc = torch.zeros(max(3 * (c1 - c0), 3), dtype=torch.int64, device=dev)
+        prof = profile_partitioned(loop, ws, group, jp, exchange, chunk_iters, cc_loc)
+        cc = torch.zeros(3 * nck, dtype=torch.int64, device=dev)
+        cc[3 * c0:3 * c1] = cc_loc[:3 * (c1 - c0)]
+        if world > 1:
+            dist.all_reduce(cc, group=group)
+        mark("profile")
+        tasks, conf = jp.jp_plan_tasks(full, cc.cpu(), chunk_iters, ws, tau_high)
+        ccl = cc.cpu().tolist()
     lv = _levels(conf, len(tasks))
     chunks, stolen = jp.jp_plan_stealing(tasks, world, chunk_iters, speed, speed_tls)
     task_of = {}
     for t, (s, e2, _) in enumerate(tasks):
         task_of[(s, e2)] = t
-    ccl = cc.cpu().tolist()
     tls_stats = {"committed": 0, "executed": 0, "windows": 0, "violations": 0}
     mine = {"chunks": 0, "iters": 0}
     mark("plan")

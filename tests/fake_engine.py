@@ -271,6 +271,19 @@ def jp_plan_tasks(loop, chunk_counts, chunk_iters, ws, tau_high=0.999):
     return [tuple(x) for x in tasks], conf
 
 
+def jp_profile_plan_tasks(loop, chunk_iters, ws, tau_high=0.999):
+    """jp.h jp_profile_plan_tasks: this rank's own profile of the whole loop (its
+    full replica) with per-chunk counts, then the plan -- composed from the
+    definitions above."""
+    nck = -(-loop.n // chunk_iters)
+    cc = torch.zeros(max(3 * nck, 3), dtype=torch.int64)
+    jp_profile_stamp(loop, ws)
+    prof = jp_profile_classify(loop, ws, chunk_iters=chunk_iters, chunk_counts=cc)
+    ccl = cc.tolist()[:3 * nck]
+    tasks, conf = jp_plan_tasks(loop, ccl, chunk_iters, ws, tau_high)
+    return prof, ccl, tasks, conf
+
+
 def jp_export_keys(loop, ws):
     ind = _indirect(loop)
     t = loop.tensors

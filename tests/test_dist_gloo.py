@@ -106,8 +106,9 @@ def _jobs(world):
         share += [("share", c, "owner") for c in ("c1_5", "c4", "c5tail", "c5head")]
     else:
         share += [("share", "c5tail", "owner")]
-    steal = [("steal", "c5", "dense"), ("steal", "c5", "owner")] + \
-        ([("steal", "c1_5", "dense"), ("steal", "seq", "dense")] if world == 2 else [])
+    steal = [("steal", "c5", "dense"), ("steal", "c5", "owner"), ("steal", "c5", "dense+repl")] + \
+        ([("steal", "c1_5", "dense"), ("steal", "seq", "dense"), ("steal", "c5", "owner+repl"),
+          ("steal", "seq", "dense+repl")] if world == 2 else [])
     return share + steal
 
 
@@ -174,7 +175,11 @@ def _steal_case(rank, world, case, exchange, q):
         full = jp.Loop.from_workload(wl)
         ws = torch.zeros(jp.jp_workspace_bytes(full), dtype=torch.uint8)
         jd.OWNER_MIN_LEN = 0
-        res = jd.schedule_stealing(full, ws, chunk_iters=1024, exchange=exchange, engine=fe)
+        # "<exchange>+repl": every rank profiles its full replica (jp_profile_plan_tasks);
+        # otherwise the partitioned profile with C1 / C3
+        xch, _, repl = exchange.partition("+")
+        res = jd.schedule_stealing(full, ws, chunk_iters=1024, exchange=xch, engine=fe,
+                                   profile="replicated" if repl else "partitioned")
         ok = wl.A.numpy().tobytes() == A_exp.tobytes()
         q.put((rank, bool(ok), res["n_tasks"], res["n_batches"], res["rank_work"]["iters"]))
     except Exception:  # pragma: no cover
@@ -184,11 +189,14 @@ def _steal_case(rank, world, case, exchange, q):
 
 @pytest.mark.parametrize("case,world,exchange", [("c5", 2, "dense"), ("c5", 3, "dense"), ("c5", 2, "owner"),
                                                   ("c5", 3, "owner"), ("c1_5", 2, "dense"), ("seq", 2, "dense"),
-                                                  ("c5", 4, "owner")])
+                                                  ("c5", 4, "owner"), ("c5", 2, "dense+repl"),
+                                                  ("c5", 3, "dense+repl"), ("c5", 2, "owner+repl"),
+                                                  ("seq", 2, "dense+repl")])
 def test_stealing_scheme_matches_oracle(case, world, exchange):
     """Multi-rank task stealing (dist.schedule_stealing): partitioned profile with
-    chunk counts, tasks + PDG, Alg. 1 plan, batches with C4 merges; every
-    replica ends with the oracle's sequential result."""
+    chunk counts (or, "+repl", every rank's own profile of its full replica),
+    tasks + PDG, Alg. 1 plan, batches with C4 merges; every replica ends with the
+    oracle's sequential result."""
     out = run_world(world, "steal", case, exchange)
     assert [o[1] for o in out] == [True] * world, out
     assert sum(o[4] for o in out) == (3 * 1024 if case == "seq" else 4096)

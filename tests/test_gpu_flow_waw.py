@@ -72,6 +72,21 @@ def test_random_raw_war_waw(seed, dtype):
     assert res["prof"]["war_iters"] > 0 and res["prof"]["waw_iters"] > 0
 
 
+@pytest.mark.parametrize("frac", [0.5, 0.9])
+def test_inplace_mix(frac):
+    """In-place updates (r[i] == w[i]: one access record for read and write in the
+    profile) mixed with random reads and duplicate writes: path 9 reads the
+    also-read records as reads."""
+    n = (1 << 20) + 11
+    g = np.random.default_rng(17)
+    w = g.integers(0, n, n).astype(np.int32)
+    r = np.where(g.random(n) < frac, w, g.integers(0, n, n)).astype(np.int32)
+    A = torch.from_numpy(g.integers(-2**31, 2**31, size=n, dtype=np.int64).astype(np.int32))
+    wl = synth.Workload("inplace_mix", O.OP_ADD_C, O.I32, n, A, r=torch.from_numpy(r), w=torch.from_numpy(w), c0=5)
+    res = run_and_check(wl)
+    assert res["prof"]["waw_iters"] > 0, res["prof"]
+
+
 def _war_only(n: int, k: int, seed: int = 5):
     """w[i] = r[i-1] (every write lands on an address an EARLIER iteration read,
     no earlier writer: WAR on the window-start value, no WAW), and k iterations

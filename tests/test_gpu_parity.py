@@ -1172,11 +1172,18 @@ def _bucket_cases():
                                         r=torch.from_numpy(g.integers(0, n, n).astype(np.int32)),
                                         w=torch.from_numpy(g.integers(0, n, n).astype(np.int32)),
                                         X=torch.from_numpy(g.standard_normal(n).astype(np.float32)), c0=1.1)))
+    # in-place updates (r[i] == w[i], one access record for both) for a random
+    # half of the iterations, random reads and duplicate writes for the rest
+    wm = g.integers(0, n, n).astype(np.int32)
+    rm = np.where(g.random(n) < 0.5, wm, g.integers(0, n, n)).astype(np.int32)
+    out.append(("inplace_mix", synth.Workload("inplace_mix", O.OP_ADD_C, O.I32, n,
+                                              torch.from_numpy(g.integers(0, 99, n).astype(np.int32)),
+                                              r=torch.from_numpy(rm), w=torch.from_numpy(wm), c0=3)))
     return out
 
 
 @pytest.mark.parametrize("buckets", ["1", "0"])
-@pytest.mark.parametrize("case", range(5))
+@pytest.mark.parametrize("case", range(6))
 def test_schedule_bucket_profile(case, buckets, monkeypatch):
     """jp_schedule's profile of a large A by address buckets (jp_bucket.cu) --
     and, with JP_PROFILE_BUCKETS=0, the stamp/classify profile it replaces --
