@@ -711,18 +711,19 @@ def partitioned_config5(jp, dev, st, world, rank, steps):
     wl.A.copy_(A0)
     barrier(world)
     ph = jd.schedule_stealing(full, ws, chunk_iters=65536, timings=True, force_ranks=True)["phases"]
-    forced_ms = None
+    forced_ms = {}
     if world == 1:
-        fts = []
-        for k in range(6):
-            wl.A.copy_(A0)
-            torch.cuda.synchronize()
-            t0 = time.perf_counter()
-            jd.schedule_stealing(full, ws, chunk_iters=65536, force_ranks=True)
-            torch.cuda.synchronize()
-            if k >= 1:
-                fts.append(time.perf_counter() - t0)
-        forced_ms = statistics.median(fts) * 1e3
+        for prof_kind in ("replicated", "partitioned"):
+            fts = []
+            for k in range(6):
+                wl.A.copy_(A0)
+                torch.cuda.synchronize()
+                t0 = time.perf_counter()
+                jd.schedule_stealing(full, ws, chunk_iters=65536, force_ranks=True, profile=prof_kind)
+                torch.cuda.synchronize()
+                if k >= 1:
+                    fts.append(time.perf_counter() - t0)
+            forced_ms[prof_kind] = statistics.median(fts) * 1e3
     # device-side stealing (jp_run_priv_claim): chunks claimed at run time
     dts, dres = [], {"rank_work": "skipped: CUDA-IPC rows turned off (JP_BENCH_IPC=0)"}
     try:
