@@ -182,8 +182,11 @@ typedef struct {
                                    one-CTA schedule; 5 / 6 on-chip recovery on a
                                    cluster / on every SM; 7 one-warp program order
                                    for mode C; 8 on-chip recovery in one window;
-                                   9 the same over a loop with WAR / WAW
-                                   (reading B14, jp_schedule only: every
+                                   9 the same over an ADD_C or SAXPY loop
+                                   with WAR / WAW (SAXPY with duplicate
+                                   writes: a scatter-add whose writers of one
+                                   address chain; reading B14, jp_schedule
+                                   only: every
                                    violator fed from the LAST earlier writer of
                                    its address, from a per-iteration shadow slot
                                    in region 8, its index in region 7; last

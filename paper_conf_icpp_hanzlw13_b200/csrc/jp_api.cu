@@ -2213,11 +2213,12 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
     res->task_mode_iters[JP_MODE_TLS] += L->n;
     return JP_OK;
   }
-  // an ADD_C TLS loop WITH WAR / WAW, profiled by address buckets: the last
+  // an ADD_C or SAXPY TLS loop WITH WAR / WAW, profiled by address buckets: the last
   // earlier writer of every raw read from the records still in place, then one
   // window over the whole loop (path 9, reading B14, jp_tls_flow.cu); the
   // windowed paths stay for what the last-writer pass cannot hold
-  if (bucket && res->mode == JP_MODE_TLS && j.op == JP_OP_ADD_C && (p.war_iters > 0 || p.waw_iters > 0) &&
+  if (bucket && res->mode == JP_MODE_TLS && (j.op == JP_OP_ADD_C || j.op == JP_OP_SAXPY) &&
+      (p.war_iters > 0 || p.waw_iters > 0) &&
       c.tls_recovery == 0 && c.tls_path == 0 && c.tls_window == 0 && !getenv("JP_TLS_NO_FLOW")) {
     int64_t *hd = at<int64_t>(ws, lg, R_HEADER);
     auto *pred = at<int32_t>(ws, lg, R_TLS_S_A);

@@ -463,6 +463,7 @@ struct PredOut {
   uint32_t *pub, *now, *later;    // [nw] each, zeroed by the caller
   int64_t *hdr;                   // H_PRED_FAIL, H_PRED_SEG
   uint32_t *redo;                 // [B] bucket left to the big tier
+  int all_read;                   // SAXPY: every write record also reads its address (Y[w])
 };
 
 template <bool BIG>
@@ -545,7 +546,7 @@ __device__ __forceinline__ void pred_bucket(int b, const uint32_t *base, const u
   __syncthreads();
   // reads: the largest writer below i in the address's list
   sweep([&](unsigned long long x) {
-    if (!rec_reads(x)) return;
+    if (!rec_reads(x) && !O.all_read) return;
     const uint32_t i = (uint32_t)x, al = (uint32_t)(x >> 32) & (kBSpan - 1);
     const uint32_t p0 = al ? cur[al - 1] : 0u, p1 = cur[al];
     if (p0 == p1) return;   // an address nobody writes
@@ -736,7 +737,7 @@ cudaError_t launch_prof_bucket(const Job &j, void *ws, const Layout &lo, uint32_
 cudaError_t launch_prof_pred(const Job &j, void *ws, const Layout &lo, int32_t *pred, uint32_t *bits,
                              unsigned long long *V, cudaStream_t st) {
   BkPlan P;
-  if (j.op != JP_OP_ADD_C || !plan(j, ws, lo, P)) return cudaErrorInvalidValue;
+  if ((j.op != JP_OP_ADD_C && j.op != JP_OP_SAXPY) || !plan(j, ws, lo, P)) return cudaErrorInvalidValue;
   const int64_t nw = (j.d.n + 31) / 32;
   cudaError_t e = cudaMemsetAsync(bits, 0, 3 * 4 * (size_t)nw, st);
   // redo flags in the per-tile offsets (P.cnt: the scatter was their last reader)
@@ -746,7 +747,7 @@ cudaError_t launch_prof_pred(const Job &j, void *ws, const Layout &lo, int32_t *
   if (e == cudaSuccess)
     e = set_smem_once((const void *)k_bk_pred_big, (int)kPredSmemB);
   if (e != cudaSuccess) return e;
-  PredOut O{pred, V, bits, bits + nw, bits + 2 * nw, at<int64_t>(ws, lo, R_HEADER), P.cnt};
+  PredOut O{pred, V, bits, bits + nw, bits + 2 * nw, at<int64_t>(ws, lo, R_HEADER), P.cnt, j.op == JP_OP_SAXPY};
   k_bk_pred<<<P.v.B, 512, kPredSmemS, st>>>(P.base, P.tot, P.rec, O);
   k_bk_pred_big<<<std::min(P.v.B, num_sms()), 1024, kPredSmemB, st>>>(P.v.B, P.base, P.tot, P.rec, O);
   note_launch(2);

@@ -211,11 +211,14 @@ static cudaError_t run_flow(const Job &j, const uint32_t *graw, const uint32_t *
 struct FlowSetW {
   int32_t r[kFlowK], w[kFlowK], pr[kFlowK];
   uint32_t f[kFlowK];   // the iteration's bits: raw 1, publish 2, commit now 4, commit later 8
-  uint32_t x[kFlowK];
+  uint32_t x[kFlowK];   // the exposed read of A (non-violators): A[r] (ADD_C), Y[w] (SAXPY)
+  uint32_t xs[kFlowK];  // SAXPY: X[r] (read-only, gathered for every iteration)
 };
 constexpr uint32_t kFRaw = 1, kFPub = 2, kFNow = 4, kFLater = 8;
 
-template <int DT>
+// OP: ADD_C (A[w] = A[r] + c0) or SAXPY (Y[w] = c0*X[r] + Y[w], its exposed read
+// is of the address it writes: a scatter-add whose duplicate writes chain)
+template <int OP, int DT>
 struct FlowW {
   DLoop L;
   const uint32_t *graw, *gpub, *gnow, *glater;
@@ -244,8 +247,16 @@ struct FlowW {
   }
   __device__ __forceinline__ void gather(uint32_t base, FlowSetW &s) const {
 #pragma unroll
-    for (int k = 0; k < kFlowK; k++)
-      if (act(base, k) && !(s.f[k] & kFRaw)) s.x[k] = __ldcg(L.A + s.r[k]);
+    for (int k = 0; k < kFlowK; k++) {
+      if (!act(base, k)) continue;
+      if constexpr (OP == JP_OP_SAXPY) s.xs[k] = __ldcg(L.X + s.r[k]);
+      if (!(s.f[k] & kFRaw)) s.x[k] = __ldcg(L.A + (OP == JP_OP_SAXPY ? s.w[k] : s.r[k]));
+    }
+  }
+  // the body's value from the exposed read a (of A / Y)
+  __device__ __forceinline__ uint32_t body(const FlowSetW &s, int k, uint32_t a) const {
+    if constexpr (OP == JP_OP_SAXPY) return op_add<DT>(op_mul<DT>(L.c0, s.xs[k]), a);
+    else return op_add<DT>(a, L.c0);
   }
   __device__ __forceinline__ void commit(const FlowSetW &s, uint32_t base, int k, uint32_t v) const {
     if (s.f[k] & kFNow) __stcg(L.A + s.w[k], v);
@@ -258,7 +269,7 @@ struct FlowW {
     for (int k = 0; k < kFlowK; k++) {
       if (!act(base, k)) continue;
       if (s.f[k] & kFRaw) pend |= 1u << k;
-      else commit(s, base, k, op_add<DT>(s.x[k], L.c0));
+      else commit(s, base, k, body(s, k, s.x[k]));
     }
     viol += __popc(pend);
     long long spins = 0;
@@ -269,7 +280,7 @@ struct FlowW {
           unsigned long long v;
           asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(v) : "l"(V + s.pr[k]) : "memory");
           if ((v >> 32) == 1ull) {
-            commit(s, base, k, op_add<DT>((uint32_t)v, L.c0));
+            commit(s, base, k, body(s, k, (uint32_t)v));
             pend &= ~(1u << k);
           }
         }
@@ -282,13 +293,13 @@ struct FlowW {
   }
 };
 
-template <int DT>
+template <int OP, int DT>
 __global__ void __launch_bounds__(kFlowT, JP_FLOW_MINB) k_tls_flow_waw(DLoop L, const uint32_t *graw, const int32_t *pred,
                                                            const uint32_t *bits, unsigned long long *V,
                                                            int64_t *stats, const int64_t *gate) {
   if (gate && gate[H_PRED_FAIL] != 0) return;   // grid-uniform: no barrier is entered
   const uint32_t nw = (uint32_t)((L.n + 31) / 32);
-  FlowW<DT> F;
+  FlowW<OP, DT> F;
   F.L = L; F.graw = graw; F.pred = pred; F.V = V;
   F.gpub = bits; F.gnow = bits + nw; F.glater = bits + 2 * nw;
   F.G = gridDim.x * (uint32_t)kFlowT;
@@ -326,11 +337,11 @@ __global__ void __launch_bounds__(kFlowT, JP_FLOW_MINB) k_tls_flow_waw(DLoop L, 
   }
 }
 
-template <int DT>
+template <int OP, int DT>
 static cudaError_t run_flow_waw(const Job &j, const uint32_t *graw, const int32_t *pred, const uint32_t *bits,
                                 unsigned long long *V, int64_t *stats, const int64_t *gate, cudaStream_t st) {
-  int maxb = 0;
-  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&maxb, (const void *)k_tls_flow_waw<DT>, kFlowT, 0);
+  static int maxb = 0;   // (one device model per process: B200)
+  if (maxb < 1) cudaOccupancyMaxActiveBlocksPerMultiprocessor(&maxb, (const void *)k_tls_flow_waw<OP, DT>, kFlowT, 0);
   if (maxb < 1) return cudaErrorInvalidConfiguration;
   int grid = num_sms() * maxb;
   const int64_t need = (j.d.n + kFlowT - 1) / kFlowT;
@@ -338,16 +349,22 @@ static cudaError_t run_flow_waw(const Job &j, const uint32_t *graw, const int32_
   DLoop d = j.d;
   void *args[] = {&d, &graw, &pred, &bits, &V, &stats, &gate};
   note_launch();
-  return cudaLaunchCooperativeKernel((const void *)k_tls_flow_waw<DT>, dim3(grid), dim3(kFlowT), args, 0, st);
+  return cudaLaunchCooperativeKernel((const void *)k_tls_flow_waw<OP, DT>, dim3(grid), dim3(kFlowT), args, 0, st);
 }
 
 cudaError_t launch_tls_flow_waw(const Job &j, const uint32_t *graw, const int32_t *pred, const uint32_t *bits,
                                 unsigned long long *V, int64_t *stats, const int64_t *gate, cudaStream_t st) {
   cudaMemsetAsync(stats, 0, 4 * sizeof(int64_t), st);
   if (j.d.n == 0) return launch_check();
-  if (j.op != JP_OP_ADD_C) return cudaErrorInvalidValue;
-  cudaError_t e = j.dt == JP_F32 ? run_flow_waw<JP_F32>(j, graw, pred, bits, V, stats, gate, st)
-                                 : run_flow_waw<JP_I32>(j, graw, pred, bits, V, stats, gate, st);
+  cudaError_t e;
+  if (j.op == JP_OP_ADD_C)
+    e = j.dt == JP_F32 ? run_flow_waw<JP_OP_ADD_C, JP_F32>(j, graw, pred, bits, V, stats, gate, st)
+                       : run_flow_waw<JP_OP_ADD_C, JP_I32>(j, graw, pred, bits, V, stats, gate, st);
+  else if (j.op == JP_OP_SAXPY)
+    e = j.dt == JP_F32 ? run_flow_waw<JP_OP_SAXPY, JP_F32>(j, graw, pred, bits, V, stats, gate, st)
+                       : run_flow_waw<JP_OP_SAXPY, JP_I32>(j, graw, pred, bits, V, stats, gate, st);
+  else
+    return cudaErrorInvalidValue;
   if (e != cudaSuccess) return e;
   return launch_check();
 }

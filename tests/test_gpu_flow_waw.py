@@ -87,6 +87,36 @@ def test_inplace_mix(frac):
     assert res["prof"]["waw_iters"] > 0, res["prof"]
 
 
+@pytest.mark.parametrize("dtype", [0, 1], ids=["i32", "f32"])
+@pytest.mark.parametrize("dup", [0.3, 0.7, 0.9])
+def test_saxpy_scatter_add(dtype, dup):
+    """SAXPY with duplicate indirect writes, Y[w[i]] = c0*X[r[i]] + Y[w[i]] (a
+    scatter-add: the writers of one address form a dependence chain, raw = waw):
+    path 9 feeds every later writer from its address's previous writer.  At
+    dup = 0.7 a bucket of 8192 addresses gets ~27K writes (the one-CTA-per-SM
+    tier of the last-writer pass); at 0.9 ~82K, more than that tier holds: the
+    windowed paths run instead (same bytes)."""
+    n = (1 << 20) + 29
+    g = np.random.default_rng(23 + int(10 * dup))
+    m = int(n * (1 - dup)) + 1       # fewer distinct targets -> more duplicates
+    w = g.integers(0, m, n).astype(np.int32)
+    r = g.integers(0, n, n).astype(np.int32)
+    if dtype == O.I32:
+        Y = torch.from_numpy(g.integers(-2**31, 2**31, size=n, dtype=np.int64).astype(np.int32))
+        X = torch.from_numpy(g.integers(-2**31, 2**31, size=n, dtype=np.int64).astype(np.int32))
+        c0 = 3
+    else:
+        Y = torch.from_numpy(((g.integers(0, 2**23, size=n) * 2.0**-22) - 1).astype(np.float32))
+        X = torch.from_numpy(((g.integers(0, 2**23, size=n) * 2.0**-22) - 1).astype(np.float32))
+        c0 = float(np.float32(1.1))
+    wl = synth.Workload("scatter_add", O.OP_SAXPY, dtype, n, Y, r=torch.from_numpy(r), w=torch.from_numpy(w),
+                        X=X, c0=c0)
+    res = run_and_check(wl, expect_path=9 if dup < 0.8 else None)
+    assert res["prof"]["raw_iters"] == res["prof"]["waw_iters"] > 0, res["prof"]
+    if dup > 0.8:
+        assert res["tls_path"] != 9, res
+
+
 def _war_only(n: int, k: int, seed: int = 5):
     """w[i] = r[i-1] (every write lands on an address an EARLIER iteration read,
     no earlier writer: WAR on the window-start value, no WAW), and k iterations
