@@ -430,6 +430,26 @@ def modes_sweep(jp, dev, st):
             waw.append(row)
             del wl, ws, L, A0
     out["config3_waw"] = waw
+    # SAXPY with duplicate indirect writes (a scatter-add, raw = waw: the writers
+    # of one address chain), N = 2^24 fp32: path 9 through jp_schedule
+    sax = []
+    for dup in (0.3, 0.7):
+        g = torch.Generator(device="cpu").manual_seed(1017)
+        n = 1 << 24
+        m = int(n * (1 - dup)) + 1
+        w = torch.randint(0, m, (n,), generator=g, dtype=torch.int32).to(dev)
+        r = torch.randint(0, n, (n,), generator=g, dtype=torch.int32).to(dev)
+        Y = (torch.randint(0, 1 << 23, (n,), generator=g).to(torch.float32) * 2.0 ** -22 - 1).to(dev)
+        X = (torch.randint(0, 1 << 23, (n,), generator=g).to(torch.float32) * 2.0 ** -22 - 1).to(dev)
+        Y0 = Y.clone()
+        L = jp.Loop(jp.JP_OP_SAXPY, jp.JP_F32, n, Y, r=r, w=w, X=X, c0=1.1)
+        ws = jp.workspace(L)
+        res, ms = timed(lambda: jp.jp_schedule(L, ws, stream=st), Y, Y0)
+        sax.append({"dup_frac": dup, "n": n, "mode": res["mode_name"], "ms": ms, "committed_per_s": n / (ms * 1e-3),
+                    "raw_iters": res["prof"]["raw_iters"], "tls_path": names.get(res["tls_path"], "?"),
+                    "windows": res["tls"]["windows"]})
+        del L, ws, Y, Y0, X, r, w
+    out["saxpy_scatter_add"] = sax
     out["crossover"] = crossover_sweep(jp, dev, st)
     # config 4: privatized.  The whole jp_schedule call (what a user runs: reading
     # B11 decides privatized without a profile, the s indices are checked on the
