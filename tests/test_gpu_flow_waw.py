@@ -185,3 +185,25 @@ def test_repeat_same_workspace():
     res = jp.jp_schedule(L1, ws)
     torch.cuda.synchronize()
     assert res["tls_path"] == 8 and equal_bytes(g1.A, A1), res
+
+
+@pytest.mark.parametrize("split", [2, 3])
+def test_ranges_of_config3_waw(split):
+    """config3_waw run as consecutive ranges (iter_base = ident_off = the range
+    start), each through jp_schedule on the shared arrays: every range is a loop of
+    its own (path 9 when it still has raw reads inside it, reads of earlier ranges'
+    writes see A); the final A is the sequential one."""
+    n = (1 << 21) + 10
+    wl = synth.config3_waw(0.05, n=n, delta=1024)
+    _, A, _ = O.run_seq(to_oracle(wl))
+    g = wl.to(DEV)
+    full = jp.Loop.from_workload(g)
+    cuts = [n * k // split for k in range(split + 1)]
+    paths = []
+    for b, e in zip(cuts[:-1], cuts[1:]):
+        part = full.range(b, e)
+        res = jp.jp_schedule(part, jp.workspace(part))
+        torch.cuda.synchronize()
+        paths.append(res["tls_path"])
+    assert equal_bytes(g.A, A), first_diff(g.A, A)
+    assert 9 in paths, paths
