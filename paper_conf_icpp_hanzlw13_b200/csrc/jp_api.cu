@@ -2247,7 +2247,10 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
       res->task_mode_iters[JP_MODE_TLS] += L->n;
       return JP_OK;
     }
-    clean &= ~1;   // region 7 now holds the pass's tables; V is untouched (the kernel exited)
+    // the pass gave up: region 7 holds its tables and V some cleared slots (the
+    // kernel exited at its gate); the windowed paths reset both themselves
+    // (clean bit 1 off; bit 2 -- V all zero -- was never set with the bucket profile)
+    clean &= ~1;
   }
   return run_mode(L, j, res->mode, &p, c, ws, ws_bytes, res, st, gfuse && p.waw_iters == 0, clean,
                   have_dist ? dist : nullptr);
