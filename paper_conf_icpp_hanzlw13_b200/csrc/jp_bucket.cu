@@ -108,7 +108,9 @@ __device__ __forceinline__ void for_tile(const BkView &V, bool vec, F &&f) {
   }
 }
 
-// cnt[t * B + b] = accesses of tile t into bucket b; out-of-range indices counted into *bad
+// cnt[t * B + b] = records of tile t in bucket b: writes (an also-read record
+// included) in the low 16 bits, pure reads << 16 (a tile holds at most 16384 of
+// each); out-of-range indices counted into *bad
 template <int OP>
 __global__ void __launch_bounds__(kBThreads, 2) k_bk_count(BkView V, int vec, uint32_t *cnt, int64_t *bad) {
   if (gated(V.gate)) return;
@@ -133,7 +135,7 @@ __global__ void __launch_bounds__(kBThreads, 2) k_bk_count(BkView V, int vec, ui
           const uint32_t c = (uint32_t)q4(r4, k);
           const bool okc = c < V.lenA;
           nbad += !okc;
-          if (c != a) atomicAdd(&h[okc ? c >> kBShift : 0], 1u);   // (c == a: one record for both)
+          if (c != a) atomicAdd(&h[okc ? c >> kBShift : 0], 1u << 16);   // (c == a: one record for both)
           if (okc) { mn = min(mn, c); mx = max(mx, c); }
         }
       }
@@ -155,31 +157,45 @@ __global__ void __launch_bounds__(kBThreads, 2) k_bk_count(BkView V, int vec, ui
   for (int b = threadIdx.x; b < V.B; b += kBThreads) row[b] = h[b];
 }
 
-// per bucket: exclusive prefix over the tiles (in place) and the bucket total.
+// per bucket: exclusive prefix over the tiles (in place) of the records kept and
+// the bucket total.  A bucket no iteration writes drops its pure reads (a read
+// with no writer of its address is neither raw nor the first read of a written
+// address: it changes no count, guide bit or table of the profile): wflag[b].
 // Block = 32 buckets (one per lane) x 32 tile segments (one per warp).
 __global__ void __launch_bounds__(1024) k_bk_scan_tiles(uint32_t *cnt, int T, int B, uint32_t *tot,
-                                                         const int64_t *gate) {
+                                                         uint32_t *wflag, const int64_t *gate) {
   if (gated(gate)) return;
-  __shared__ uint32_t part[32][33];
+  __shared__ uint32_t part_w[32][33], part_r[32][33];
   const int lane = threadIdx.x & 31, seg = threadIdx.x >> 5;
   const int b = blockIdx.x * 32 + lane;
   const int per = (T + 31) / 32, t0 = seg * per, t1 = min(T, t0 + per);
-  uint32_t s = 0;
+  uint32_t sw = 0, sr = 0;
   if (b < B)
 #pragma unroll 8
-    for (int t = t0; t < t1; t++) s += cnt[(size_t)t * B + b];
-  part[seg][lane] = s;
+    for (int t = t0; t < t1; t++) {
+      const uint32_t c = cnt[(size_t)t * B + b];
+      sw += c & 0xFFFFu;
+      sr += c >> 16;
+    }
+  part_w[seg][lane] = sw;
+  part_r[seg][lane] = sr;
   __syncthreads();
+  uint32_t allw = 0;
+  for (int k = 0; k < 32; k++) allw += part_w[k][lane];
+  const bool keep = allw > 0;
   uint32_t run = 0;
-  for (int k = 0; k < seg; k++) run += part[k][lane];
+  for (int k = 0; k < seg; k++) run += part_w[k][lane] + (keep ? part_r[k][lane] : 0u);
   if (b < B) {
 #pragma unroll 8
     for (int t = t0; t < t1; t++) {
-      const uint32_t v = cnt[(size_t)t * B + b];
+      const uint32_t c = cnt[(size_t)t * B + b];
       cnt[(size_t)t * B + b] = run;
-      run += v;
+      run += (c & 0xFFFFu) + (keep ? c >> 16 : 0u);
     }
-    if (seg == 31) tot[b] = run;
+    if (seg == 31) {
+      tot[b] = run;
+      wflag[b] = keep ? 1u : 0u;
+    }
   }
 }
 
@@ -219,7 +235,8 @@ __global__ void __launch_bounds__(1024) k_bk_scan_buckets(const uint32_t *tot, i
 // and cursors (B each), the global start of this tile's run in every bucket.
 template <int OP>
 __global__ void __launch_bounds__(kBThreads) k_bk_scatter(BkView V, int vec, const uint32_t *off, const uint32_t *tot,
-                                                         const uint32_t *base, unsigned long long *rec) {
+                                                         const uint32_t *base, const uint32_t *wflag,
+                                                         unsigned long long *rec) {
   if (gated(V.gate)) return;
   // staging: 6 bytes per record -- il | address in the bucket << 14 | write << 31,
   // and the bucket (16 bits) -- so that a 16384-iteration tile fits one SM
@@ -229,6 +246,7 @@ __global__ void __launch_bounds__(kBThreads) k_bk_scatter(BkView V, int vec, con
   uint32_t *lpos = reinterpret_cast<uint32_t *>(stb + 2 * kTile);       // [B + 1] local exclusive starts
   uint32_t *cur = lpos + V.B + 1;                              // [B]
   uint32_t *gpos = cur + V.B;                                  // [B] global start of this tile's run
+  uint8_t *wf = reinterpret_cast<uint8_t *>(gpos + V.B);       // [B] the bucket is written (else drop pure reads)
   __shared__ uint32_t wsum[kBThreads / 32];
   const int t = blockIdx.x, B = V.B;
   const uint32_t i0 = (uint32_t)t << kTShift;
@@ -241,6 +259,7 @@ __global__ void __launch_bounds__(kBThreads) k_bk_scatter(BkView V, int vec, con
     const uint32_t c = (nxt ? nxt[b] : tot[b]) - row[b];
     cur[b] = c;   // (count, for the scan below)
     gpos[b] = base[b] + row[b];
+    wf[b] = (uint8_t)wflag[b];
     s += c;
   }
   uint32_t x = s;
@@ -276,19 +295,21 @@ __global__ void __launch_bounds__(kBThreads) k_bk_scatter(BkView V, int vec, con
     bool same[4];
 #pragma unroll
     for (int k = 0; k < 4; k++) same[k] = OP == JP_OP_ADD_C && a[2 * k] == a[2 * k + 1];
+    // skip[m]: a read folded into its iteration's write record, or a pure read of
+    // a bucket nobody writes (dropped, see k_bk_scan_tiles)
+    bool skip[kA];
 #pragma unroll
     for (int m = 0; m < kA; m++) {
       if (a[m] >= V.lenA) a[m] = 0;   // (the count pass filed it under bucket 0 too)
       const int k = OP == JP_OP_ADD_C ? m >> 1 : m;
-      const bool skip = OP == JP_OP_ADD_C && (m & 1) && same[k];
-      pos[m] = k < kn && !skip ? atomicAdd(&cur[a[m] >> kBShift], 1u) : 0u;
+      skip[m] = OP == JP_OP_ADD_C && (m & 1) && (same[k] || !wf[a[m] >> kBShift]);
+      pos[m] = k < kn && !skip[m] ? atomicAdd(&cur[a[m] >> kBShift], 1u) : 0u;
     }
 #pragma unroll
     for (int m = 0; m < kA; m++) {
       const int k = OP == JP_OP_ADD_C ? m >> 1 : m;
       const bool wr = OP == JP_OP_ADD_C ? (m & 1) == 0 : true;
-      const bool skip = OP == JP_OP_ADD_C && (m & 1) && same[k];
-      if (k < kn && !skip) {
+      if (k < kn && !skip[m]) {
         stage[pos[m]] = (uint32_t)(il0 + k) | (a[m] & (kBSpan - 1)) << kTShift | (wr ? 1u << 31 : 0u) |
                         (wr && same[k] ? 1u << 30 : 0u);
         stb[pos[m]] = (uint16_t)(a[m] >> kBShift);
@@ -643,7 +664,7 @@ namespace {
 struct BkPlan {
   BkView v;
   unsigned long long *rec;
-  uint32_t *cnt, *tot, *base;
+  uint32_t *cnt, *tot, *base, *wflag;
 };
 
 bool plan(const Job &j, void *ws, const Layout &lo, BkPlan &P) {
@@ -670,12 +691,25 @@ bool plan(const Job &j, void *ws, const Layout &lo, BkPlan &P) {
   // 256-byte alignment padding of the workspace: the span is one free piece)
   const size_t rb = lo.bytes[R_KEYS_A] ? lo.off[R_KEYS_A] + lo.bytes[R_KEYS_A] - lo.off[R_MINW_A] : 0;
   if (!lo.bytes[R_MINW_A] || rb < 8 * (size_t)nrec) return false;
-  if (lo.bytes[R_MAXRX_A] < 4 * ((size_t)T * B + 2 * (size_t)B)) return false;
+  if (lo.bytes[R_MAXRX_A] < 4 * ((size_t)T * B + 3 * (size_t)B)) return false;
+  // the scatter stages a whole tile plus three words and a flag per bucket in
+  // shared memory: len_A up to ~2.7K buckets (~22 M elements) on a 227 KB SM
+  static int smax = 0;
+  if (!smax) {
+    int dev = 0;
+    cudaGetDevice(&dev);
+    if (cudaDeviceGetAttribute(&smax, cudaDevAttrMaxSharedMemoryPerBlockOptin, dev) != cudaSuccess || smax <= 0) {
+      cudaGetLastError();
+      smax = 227 * 1024;
+    }
+  }
+  if (6 * 2 * (size_t)kTile + 4 * (3 * (size_t)B + 1) + (size_t)B + 256 > (size_t)smax) return false;
   P.v = BkView{d.r, d.w, d.n, d.ioff, (uint32_t)d.lenA, B, T, nullptr, 1, nullptr};
   P.rec = at<unsigned long long>(ws, lo, R_MINW_A);
   P.cnt = at<uint32_t>(ws, lo, R_MAXRX_A);
   P.tot = P.cnt + (size_t)T * B;
   P.base = P.tot + B;
+  P.wflag = P.base + B;
   return true;
 }
 
@@ -685,11 +719,11 @@ void run_bucket(const BkPlan &P, const DLoop &d, int64_t *hdr, BkOut O, cudaStre
   const int vec = al(d.r) && al(d.w);
   const int B = P.v.B, T = P.v.T;
   k_bk_count<OP><<<T, kBThreads, 4 * (size_t)B, st>>>(P.v, vec, P.cnt, &hdr[H_BAD]);
-  k_bk_scan_tiles<<<(B + 31) / 32, 1024, 0, st>>>(P.cnt, T, B, P.tot, P.v.gate);
+  k_bk_scan_tiles<<<(B + 31) / 32, 1024, 0, st>>>(P.cnt, T, B, P.tot, P.wflag, P.v.gate);
   k_bk_scan_buckets<<<1, 1024, 0, st>>>(P.tot, B, P.base, P.v.gate);
-  const size_t ssm = 6 * 2 * (size_t)kTile + 4 * (3 * (size_t)B + 1);
+  const size_t ssm = 6 * 2 * (size_t)kTile + 4 * (3 * (size_t)B + 1) + (size_t)B;
   set_smem_once((const void *)k_bk_scatter<OP>, (int)ssm);
-  k_bk_scatter<OP><<<T, kBThreads, ssm, st>>>(P.v, vec, P.cnt, P.tot, P.base, P.rec);
+  k_bk_scatter<OP><<<T, kBThreads, ssm, st>>>(P.v, vec, P.cnt, P.tot, P.base, P.wflag, P.rec);
   const int nch = O.cc ? (int)((d.n + O.chunk - 1) / O.chunk) : 0;
   const size_t sm = 4 * (size_t)kBSpan * (OP == JP_OP_ADD_C ? 2 : 1) + (O.cc && nch <= kSmemChunks ? 12 * (size_t)nch : 0);
   set_smem_once((const void *)k_bk_eval<OP>, (int)sm);

@@ -207,3 +207,20 @@ def test_ranges_of_config3_waw(split):
         paths.append(res["tls_path"])
     assert equal_bytes(g.A, A), first_diff(g.A, A)
     assert 9 in paths, paths
+
+
+@pytest.mark.parametrize("la_log", [23, 25])
+def test_large_A_profile_choice(la_log):
+    """A random ADD_C loop over a larger A (2^23: the address-bucket profile;
+    2^25: more buckets than the scatter's shared memory holds -> the stamp /
+    classify profile): same bytes as the oracle either way, and path 9 / the
+    windowed paths as the profile allows."""
+    n = 1 << 20
+    la = 1 << la_log
+    g = np.random.default_rng(31)
+    w = g.integers(0, la, n).astype(np.int32)
+    r = np.where(g.random(n) < 0.3, np.roll(w, 7), g.integers(0, la, n)).astype(np.int32)
+    A = torch.from_numpy(g.integers(-2**31, 2**31, size=la, dtype=np.int64).astype(np.int32))
+    wl = synth.Workload("largeA", O.OP_ADD_C, O.I32, n, A, r=torch.from_numpy(r), w=torch.from_numpy(w), c0=9)
+    res = run_and_check(wl, expect_path=None)
+    assert res["mode"] == jp.JP_MODE_TLS, res
