@@ -200,10 +200,15 @@ __global__ void __launch_bounds__(1024) k_bk_scan_tiles(uint32_t *cnt, int T, in
 }
 
 // base[b] = exclusive prefix of tot over the buckets (one CTA)
+// ... and order[]: the buckets by decreasing record count (binned by floor log2),
+// the order the one-CTA-per-bucket passes take them in, so that a few heavy
+// buckets do not form the last wave (config 5: its WAW tail's buckets hold 3x
+// the records of the others)
 __global__ void __launch_bounds__(1024) k_bk_scan_buckets(const uint32_t *tot, int B, uint32_t *base,
-                                                           const int64_t *gate) {
+                                                           uint32_t *order, const int64_t *gate) {
   if (gated(gate)) return;
   __shared__ uint32_t ws[32];
+  __shared__ uint32_t bin[33];
   const int per = (B + 1023) / 1024, b0 = threadIdx.x * per;
   uint32_t s = 0;
   for (int k = 0; k < per && b0 + k < B; k++) s += tot[b0 + k];
@@ -228,6 +233,17 @@ __global__ void __launch_bounds__(1024) k_bk_scan_buckets(const uint32_t *tot, i
     base[b0 + k] = run;
     run += tot[b0 + k];
   }
+  if (!order) return;
+  if (threadIdx.x < 33) bin[threadIdx.x] = 0;
+  __syncthreads();
+  for (int k = 0; k < per && b0 + k < B; k++) atomicAdd(&bin[32 - __clz(tot[b0 + k])], 1u);   // 0..32
+  __syncthreads();
+  if (threadIdx.x == 0) {   // exclusive starts, heaviest bin first
+    uint32_t r = 0;
+    for (int q = 32; q >= 0; q--) { const uint32_t c = bin[q]; bin[q] = r; r += c; }
+  }
+  __syncthreads();
+  for (int k = 0; k < per && b0 + k < B; k++) order[atomicAdd(&bin[32 - __clz(tot[b0 + k])], 1u)] = (uint32_t)(b0 + k);
 }
 
 // records, tile-ordered inside each bucket's segment.  Shared memory: the
@@ -337,6 +353,7 @@ struct BkOut {
   int64_t *cc;
   int64_t gbase;              // global id of local iteration 0
   int32_t *wsrc;              // nullable: wsrc[i] = the first writer of raw iteration i's read (ADD_C)
+  const uint32_t *order;      // nullable: bucket of CTA k (heaviest first)
   unsigned long long *vclr;   // nullable: V[a] = 0 at every raw read's address (the one-window TLS
                               // shadow slots a violator polls: no full clear of V needed)
 };
@@ -352,7 +369,7 @@ __global__ void __launch_bounds__(kEvalThreads) k_bk_eval(BkView V, const uint32
   uint32_t *s_cc = s_dyn + (OP == JP_OP_ADD_C ? 2 : 1) * kBSpan;
   __shared__ unsigned s_dist[32];
   __shared__ unsigned long long s_cnt[3], s_first;
-  const int b = blockIdx.x;
+  const int b = O.order ? (int)O.order[blockIdx.x] : (int)blockIdx.x;
   const int nch = O.cc ? (int)((V.n + O.chunk - 1) / O.chunk) : 0;
   const bool cc_smem = O.cc && nch <= kSmemChunks;
   for (int k = threadIdx.x; k < kBSpan; k += kEvalThreads) {
@@ -484,6 +501,7 @@ struct PredOut {
   uint32_t *pub, *now, *later;    // [nw] each, zeroed by the caller
   int64_t *hdr;                   // H_PRED_FAIL, H_PRED_SEG
   uint32_t *redo;                 // [B] bucket left to the big tier
+  const uint32_t *order;          // [B] bucket of CTA k (heaviest first)
   int all_read;                   // SAXPY: every write record also reads its address (Y[w])
 };
 
@@ -598,7 +616,7 @@ __device__ __forceinline__ void pred_bucket(int b, const uint32_t *base, const u
 
 __global__ void __launch_bounds__(512, 2) k_bk_pred(const uint32_t *base, const uint32_t *tot,
                                                     const unsigned long long *rec, PredOut O) {
-  pred_bucket<false>(blockIdx.x, base, tot, rec, O);
+  pred_bucket<false>((int)O.order[blockIdx.x], base, tot, rec, O);
 }
 // the big tier: one CTA per SM walks the buckets and redoes the marked ones
 __global__ void __launch_bounds__(1024, 1) k_bk_pred_big(int B, const uint32_t *base, const uint32_t *tot,
@@ -664,7 +682,7 @@ namespace {
 struct BkPlan {
   BkView v;
   unsigned long long *rec;
-  uint32_t *cnt, *tot, *base, *wflag;
+  uint32_t *cnt, *tot, *base, *wflag, *order;
 };
 
 bool plan(const Job &j, void *ws, const Layout &lo, BkPlan &P) {
@@ -691,7 +709,7 @@ bool plan(const Job &j, void *ws, const Layout &lo, BkPlan &P) {
   // 256-byte alignment padding of the workspace: the span is one free piece)
   const size_t rb = lo.bytes[R_KEYS_A] ? lo.off[R_KEYS_A] + lo.bytes[R_KEYS_A] - lo.off[R_MINW_A] : 0;
   if (!lo.bytes[R_MINW_A] || rb < 8 * (size_t)nrec) return false;
-  if (lo.bytes[R_MAXRX_A] < 4 * ((size_t)T * B + 3 * (size_t)B)) return false;
+  if (lo.bytes[R_MAXRX_A] < 4 * ((size_t)T * B + 4 * (size_t)B)) return false;
   // the scatter stages a whole tile plus three words and a flag per bucket in
   // shared memory: len_A up to ~2.7K buckets (~22 M elements) on a 227 KB SM
   static int smax = 0;
@@ -710,6 +728,7 @@ bool plan(const Job &j, void *ws, const Layout &lo, BkPlan &P) {
   P.tot = P.cnt + (size_t)T * B;
   P.base = P.tot + B;
   P.wflag = P.base + B;
+  P.order = P.wflag + B;
   return true;
 }
 
@@ -720,7 +739,7 @@ void run_bucket(const BkPlan &P, const DLoop &d, int64_t *hdr, BkOut O, cudaStre
   const int B = P.v.B, T = P.v.T;
   k_bk_count<OP><<<T, kBThreads, 4 * (size_t)B, st>>>(P.v, vec, P.cnt, &hdr[H_BAD]);
   k_bk_scan_tiles<<<(B + 31) / 32, 1024, 0, st>>>(P.cnt, T, B, P.tot, P.wflag, P.v.gate);
-  k_bk_scan_buckets<<<1, 1024, 0, st>>>(P.tot, B, P.base, P.v.gate);
+  k_bk_scan_buckets<<<1, 1024, 0, st>>>(P.tot, B, P.base, P.order, P.v.gate);
   const size_t ssm = 6 * 2 * (size_t)kTile + 4 * (3 * (size_t)B + 1) + (size_t)B;
   set_smem_once((const void *)k_bk_scatter<OP>, (int)ssm);
   k_bk_scatter<OP><<<T, kBThreads, ssm, st>>>(P.v, vec, P.cnt, P.tot, P.base, P.wflag, P.rec);
@@ -761,7 +780,7 @@ cudaError_t launch_prof_bucket(const Job &j, void *ws, const Layout &lo, uint32_
                                                               nck, pfx);
     note_launch();
   }
-  BkOut O{hdr, graw, gsrc, chunk, cc, j.d.base, j.op == JP_OP_ADD_C ? wsrc : nullptr,
+  BkOut O{hdr, graw, gsrc, chunk, cc, j.d.base, j.op == JP_OP_ADD_C ? wsrc : nullptr, P.order,
           j.op == JP_OP_ADD_C ? vclr : nullptr};
   if (j.op == JP_OP_ADD_C) run_bucket<JP_OP_ADD_C>(P, j.d, hdr, O, st);
   else run_bucket<JP_OP_SAXPY>(P, j.d, hdr, O, st);
@@ -781,7 +800,8 @@ cudaError_t launch_prof_pred(const Job &j, void *ws, const Layout &lo, int32_t *
   if (e == cudaSuccess)
     e = set_smem_once((const void *)k_bk_pred_big, (int)kPredSmemB);
   if (e != cudaSuccess) return e;
-  PredOut O{pred, V, bits, bits + nw, bits + 2 * nw, at<int64_t>(ws, lo, R_HEADER), P.cnt, j.op == JP_OP_SAXPY};
+  PredOut O{pred, V, bits, bits + nw, bits + 2 * nw, at<int64_t>(ws, lo, R_HEADER), P.cnt, P.order,
+            j.op == JP_OP_SAXPY};
   k_bk_pred<<<P.v.B, 512, kPredSmemS, st>>>(P.base, P.tot, P.rec, O);
   k_bk_pred_big<<<std::min(P.v.B, num_sms()), 1024, kPredSmemB, st>>>(P.v.B, P.base, P.tot, P.rec, O);
   note_launch(2);
