@@ -1356,15 +1356,6 @@ static jp_status mapped_pack_wait(MappedPack &m, unsigned long long seq, cudaStr
 }
 
 #include <chrono>
-// host-side phase trace of the schedulers (JP_HOST_TRACE=1: microseconds since the previous mark, stderr)
-static void htrace(const char *what) {
-  static const bool on = getenv("JP_HOST_TRACE") != nullptr;
-  if (!on) return;
-  thread_local auto prev = std::chrono::steady_clock::now();
-  const auto now = std::chrono::steady_clock::now();
-  fprintf(stderr, "[jp host] %-16s +%.1f us\n", what, std::chrono::duration<double, std::micro>(now - prev).count());
-  prev = now;
-}
 #define HTRACE(w) htrace(w)
 
 static jp_status task_conflicts(const Job &j, const jp_loop *L, void *ws, const Layout &lo,
@@ -2094,9 +2085,11 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
       uint32_t *g = at<uint32_t>(ws, lg, R_GUIDE);
       TinyMirror &mm = tiny_mirror();
       const unsigned long long seq = defer_static ? ++mm.seq : 0;
+      if (defer_static) *reinterpret_cast<volatile unsigned long long *>(&mm.host[21]) = seq;   // read by the kernel
       JP_CUDA(launch_prof_bucket(j, ws, lg, g, g + (L->n + 31) / 32, 0, nullptr, st, nullptr, nullptr,
                                  at<unsigned long long>(ws, lg, R_TLS_C_A), defer_static ? (int)std::min<int64_t>(L->n, 64) : 0,
-                                 defer_static ? reinterpret_cast<long long *>(mm.dev + 19) : nullptr, seq),
+                                 defer_static ? reinterpret_cast<long long *>(mm.dev + 19) : nullptr,
+                                 defer_static ? reinterpret_cast<const unsigned long long *>(mm.dev + 21) : nullptr),
               "profile (buckets)");
       clean |= 4;   // V clear at every address path 8 polls
       if (defer_static) {

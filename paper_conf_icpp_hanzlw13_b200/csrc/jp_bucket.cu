@@ -35,6 +35,8 @@
 // access is Y[w], read and written by the same iteration, so raw = war = waw =
 // "an earlier iteration wrote this address" (one write record).
 #include <algorithm>
+#include <string>
+#include <vector>
 #include "jp_host.h"
 
 namespace jp {
@@ -640,7 +642,7 @@ struct PrefixDuty {
   const int32_t *p[4];
   int m;
   long long *mir;
-  unsigned long long seq;
+  const volatile unsigned long long *seq;   // the call's sequence number (mapped host word, written before the launch)
 };
 __global__ void __launch_bounds__(256) k_bk_prep(int64_t *hdr, uint32_t *graw, uint32_t *gsrc, int64_t nw, int64_t *cc,
                                                  int64_t ncc, uint32_t *cr, int64_t nck, PrefixDuty pfx) {
@@ -658,7 +660,7 @@ __global__ void __launch_bounds__(256) k_bk_prep(int64_t *hdr, uint32_t *graw, u
       hdr[H_GATE] = ok ? 1 : 0;
       if (pfx.mir) {
         pfx.mir[0] = ok ? 1 : 0;
-        asm volatile("st.release.sys.global.u64 [%0], %1;" ::"l"(pfx.mir + 1), "l"(pfx.seq) : "memory");
+        asm volatile("st.release.sys.global.u64 [%0], %1;" ::"l"(pfx.mir + 1), "l"(*pfx.seq) : "memory");
       }
     }
   }
@@ -741,14 +743,30 @@ void run_bucket(const BkPlan &P, const DLoop &d, int64_t *hdr, BkOut O, cudaStre
   k_bk_scan_tiles<<<(B + 31) / 32, 1024, 0, st>>>(P.cnt, T, B, P.tot, P.wflag, P.v.gate);
   k_bk_scan_buckets<<<1, 1024, 0, st>>>(P.tot, B, P.base, P.order, P.v.gate);
   const size_t ssm = 6 * 2 * (size_t)kTile + 4 * (3 * (size_t)B + 1) + (size_t)B;
-  set_smem_once((const void *)k_bk_scatter<OP>, (int)ssm);
   k_bk_scatter<OP><<<T, kBThreads, ssm, st>>>(P.v, vec, P.cnt, P.tot, P.base, P.wflag, P.rec);
   const int nch = O.cc ? (int)((d.n + O.chunk - 1) / O.chunk) : 0;
   const size_t sm = 4 * (size_t)kBSpan * (OP == JP_OP_ADD_C ? 2 : 1) + (O.cc && nch <= kSmemChunks ? 12 * (size_t)nch : 0);
-  set_smem_once((const void *)k_bk_eval<OP>, (int)sm);
   k_bk_eval<OP><<<B, kEvalThreads, sm, st>>>(P.v, P.base, P.tot, P.rec, O);
-  note_launch(5);
 }
+// the dynamic shared memory of the scatter and eval kernels, set before any launch
+// (and before a stream capture)
+template <int OP>
+void prepare_bucket(const BkPlan &P, const BkOut &O, const DLoop &d) {
+  const int B = P.v.B;
+  set_smem_once((const void *)k_bk_scatter<OP>, (int)(6 * 2 * (size_t)kTile + 4 * (3 * (size_t)B + 1) + (size_t)B));
+  const int nch = O.cc ? (int)((d.n + O.chunk - 1) / O.chunk) : 0;
+  set_smem_once((const void *)k_bk_eval<OP>, (int)(4 * (size_t)kBSpan * (OP == JP_OP_ADD_C ? 2 : 1) +
+                                                   (O.cc && nch <= kSmemChunks ? 12 * (size_t)nch : 0)));
+}
+
+// The profile's six launches as one CUDA graph per argument set (a call with the
+// same loop, workspace and outputs replays it): the host issues one launch instead
+// of six (~4-5 us of host time each, which left the GPU idle between the first
+// kernels).  Captured on a per-thread side stream, launched into the caller's.
+struct BkGraph {
+  std::string key;
+  cudaGraphExec_t exec;
+};
 }  // namespace
 
 bool bucket_profile_ok(const Job &j, void *ws, const Layout &lo) {
@@ -758,10 +776,12 @@ bool bucket_profile_ok(const Job &j, void *ws, const Layout &lo) {
 
 cudaError_t launch_prof_bucket(const Job &j, void *ws, const Layout &lo, uint32_t *graw, uint32_t *gsrc,
                                int64_t chunk, int64_t *cc, cudaStream_t st, int32_t *wsrc, uint32_t *crange,
-                               unsigned long long *vclr, int sample_m, long long *mir, unsigned long long seq) {
+                               unsigned long long *vclr, int sample_m, long long *mir,
+                               const unsigned long long *seq) {
   BkPlan P;
   if (!plan(j, ws, lo, P)) return cudaErrorInvalidValue;
   PrefixDuty pfx{{j.d.r, j.d.r2, j.d.w, j.d.s}, sample_m, mir, seq};
+  if (sample_m > 0 && !seq) return cudaErrorInvalidValue;
   if (sample_m > 0) P.v.gate = &at<int64_t>(ws, lo, R_HEADER)[H_GATE];
   static_assert(kTile == kBucketTile, "jp_host.h kBucketTile");
   int64_t nck = 0;
@@ -773,18 +793,62 @@ cudaError_t launch_prof_bucket(const Job &j, void *ws, const Layout &lo, uint32_
   int64_t *hdr = at<int64_t>(ws, lo, R_HEADER);
   const int64_t nw = (j.d.n + 31) / 32;
   const int64_t ncc = cc ? 3 * ((j.d.n + chunk - 1) / chunk) : 0;
-  {
-    int64_t m = std::max<int64_t>(std::max<int64_t>((int64_t)(kHeaderBytes / 8), nw), std::max(ncc, nck));
-    const int64_t need = (m + 255) / 256, cap = (int64_t)num_sms() * 4;
-    k_bk_prep<<<(int)(need < cap ? need : cap), 256, 0, st>>>(hdr, graw, gsrc, nw, cc, ncc, nck ? crange : nullptr,
-                                                              nck, pfx);
-    note_launch();
-  }
+  const int64_t mprep = std::max<int64_t>(std::max<int64_t>((int64_t)(kHeaderBytes / 8), nw), std::max(ncc, nck));
+  const int64_t need = (mprep + 255) / 256, cap = (int64_t)num_sms() * 4;
+  const int gprep = (int)(need < cap ? need : cap);
   BkOut O{hdr, graw, gsrc, chunk, cc, j.d.base, j.op == JP_OP_ADD_C ? wsrc : nullptr, P.order,
           j.op == JP_OP_ADD_C ? vclr : nullptr};
-  if (j.op == JP_OP_ADD_C) run_bucket<JP_OP_ADD_C>(P, j.d, hdr, O, st);
-  else run_bucket<JP_OP_SAXPY>(P, j.d, hdr, O, st);
-  return launch_check();
+  if (j.op == JP_OP_ADD_C) prepare_bucket<JP_OP_ADD_C>(P, O, j.d);
+  else prepare_bucket<JP_OP_SAXPY>(P, O, j.d);
+  auto issue = [&](cudaStream_t s) {
+    k_bk_prep<<<gprep, 256, 0, s>>>(hdr, graw, gsrc, nw, cc, ncc, nck ? crange : nullptr, nck, pfx);
+    if (j.op == JP_OP_ADD_C) run_bucket<JP_OP_ADD_C>(P, j.d, hdr, O, s);
+    else run_bucket<JP_OP_SAXPY>(P, j.d, hdr, O, s);
+  };
+  note_launch(6);
+  const char *ng = getenv("JP_NO_GRAPHS");
+  if (ng && ng[0] == '1') {
+    issue(st);
+    return launch_check();
+  }
+  int dev = 0;
+  cudaGetDevice(&dev);
+  // the key: every value the six launches take, field by field (no struct padding)
+  std::string key;
+  auto put = [&](auto v) { key.append(reinterpret_cast<const char *>(&v), sizeof v); };
+  put(dev); put(j.op); put(j.dt); put(gprep); put(nck); put(ncc); put(nw);
+  put(P.v.r); put(P.v.w); put(P.v.n); put(P.v.ioff); put(P.v.lenA); put(P.v.B); put(P.v.T); put(P.v.crange);
+  put(P.v.ctiles); put(P.v.gate);
+  put(P.rec); put(P.cnt); put(P.tot); put(P.base); put(P.wflag); put(P.order);
+  put(O.hdr); put(O.graw); put(O.gsrc); put(O.chunk); put(O.cc); put(O.gbase); put(O.wsrc); put(O.order); put(O.vclr);
+  for (int q = 0; q < 4; q++) put(pfx.p[q]);
+  put(pfx.m); put(pfx.mir); put(pfx.seq);
+  put(j.d.r); put(j.d.w); put(j.d.n); put(j.d.ioff); put(j.d.base);
+  thread_local std::vector<BkGraph> cache;
+  for (const BkGraph &g : cache)
+    if (g.key == key) return cudaGraphLaunch(g.exec, st);
+  thread_local cudaStream_t cs[64] = {};
+  if (!cs[dev & 63]) {
+    cudaError_t e = cudaStreamCreateWithFlags(&cs[dev & 63], cudaStreamNonBlocking);
+    if (e != cudaSuccess) return e;
+  }
+  cudaStream_t c = cs[dev & 63];
+  cudaError_t e = cudaStreamBeginCapture(c, cudaStreamCaptureModeThreadLocal);
+  if (e != cudaSuccess) return e;
+  issue(c);
+  cudaGraph_t graph = nullptr;
+  e = cudaStreamEndCapture(c, &graph);
+  if (e != cudaSuccess) return e;
+  cudaGraphExec_t exec = nullptr;
+  e = cudaGraphInstantiate(&exec, graph, 0);
+  cudaGraphDestroy(graph);
+  if (e != cudaSuccess) return e;
+  if (cache.size() >= 16) {   // (bounded: older argument sets are dropped)
+    for (BkGraph &g : cache) cudaGraphExecDestroy(g.exec);
+    cache.clear();
+  }
+  cache.push_back({key, exec});
+  return cudaGraphLaunch(exec, st);
 }
 
 cudaError_t launch_prof_pred(const Job &j, void *ws, const Layout &lo, int32_t *pred, uint32_t *bits,

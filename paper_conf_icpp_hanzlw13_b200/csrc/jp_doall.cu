@@ -10,6 +10,8 @@
 // k_doall_generic: indirect bodies (config 1 at 0%, the config-5 head):
 //   coalesced index streams, gathered/scattered element accesses.
 #include <atomic>
+#include <chrono>
+#include <cstdio>
 #include <cstdlib>
 #include <cstring>
 #include <mutex>
@@ -17,6 +19,16 @@
 #include "jp_host.h"
 
 namespace jp {
+
+// host-side phase trace of the schedulers (JP_HOST_TRACE=1: microseconds since the previous mark, stderr)
+void htrace(const char *what) {
+  static const bool on = getenv("JP_HOST_TRACE") != nullptr;
+  if (!on) return;
+  thread_local auto prev = std::chrono::steady_clock::now();
+  const auto now = std::chrono::steady_clock::now();
+  fprintf(stderr, "[jp host] %-16s +%.1f us\n", what, std::chrono::duration<double, std::micro>(now - prev).count());
+  prev = now;
+}
 
 cudaError_t set_smem_once(const void *fn, int bytes) {
   struct Ent { const void *fn; int dev, bytes; };

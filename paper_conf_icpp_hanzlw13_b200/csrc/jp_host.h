@@ -23,6 +23,8 @@ struct Layout {
 // device) and size: the attribute call costs about a microsecond of host time on
 // every launch otherwise (the launch-bound front of jp_schedule)
 cudaError_t set_smem_once(const void *fn, int bytes);
+// host-side phase marks (JP_HOST_TRACE=1: microseconds since the previous mark, to stderr)
+void htrace(const char *what);
 
 // Fixed-offset layout of a workspace for loop L (offsets do not depend on uses).
 Layout layout(const jp_loop *L);
@@ -95,7 +97,10 @@ cudaError_t launch_tls_flow(const Job &j, const uint32_t *graw, const uint32_t *
 cudaError_t launch_prof_bucket(const Job &j, void *ws, const Layout &lo, uint32_t *graw, uint32_t *gsrc,
                                int64_t chunk, int64_t *cc, cudaStream_t st, int32_t *wsrc = nullptr,
                                uint32_t *crange = nullptr, unsigned long long *vclr = nullptr, int sample_m = 0,
-                               long long *mir = nullptr, unsigned long long seq = 0);
+                               long long *mir = nullptr, const unsigned long long *seq = nullptr);
+// (seq: a mapped host word holding the call's sequence number, written by the
+// host before the launch -- the launches are replayed from a CUDA graph per
+// argument set, JP_NO_GRAPHS=1 issues them one by one)
 constexpr int64_t kBucketTile = 16384;   // (jp_bucket.cu's tile: chunk ranges need chunk % kBucketTile == 0)
 // after launch_prof_bucket on the same workspace (its records still in place),
 // ADD_C: the last earlier writer of every raw read -> pred[i] (raw i only), and
