@@ -1184,6 +1184,50 @@ static Job sub_job(const Job &j, int64_t s, int64_t e) {
   return k;
 }
 
+// Replay of a fixed launch sequence from a CUDA graph cached per key (the values
+// its launches take): captured once on a per-thread side stream, then launched
+// into st.  JP_NO_GRAPHS=1 issues the sequence directly.
+static cudaError_t graph_launch(const std::string &key, const std::function<cudaError_t(cudaStream_t)> &issue,
+                                cudaStream_t st) {
+  const char *ng = getenv("JP_NO_GRAPHS");
+  if (ng && ng[0] == '1') return issue(st);
+  struct Ent { std::string key; cudaGraphExec_t exec; };
+  thread_local std::vector<Ent> cache;
+  for (const Ent &e : cache)
+    if (e.key == key) return cudaGraphLaunch(e.exec, st);
+  int dev = 0;
+  cudaGetDevice(&dev);
+  thread_local cudaStream_t cs[64] = {};
+  if (!cs[dev & 63]) {
+    const cudaError_t e = cudaStreamCreateWithFlags(&cs[dev & 63], cudaStreamNonBlocking);
+    if (e != cudaSuccess) return e;
+  }
+  const cudaStream_t c = cs[dev & 63];
+  cudaError_t e = cudaStreamBeginCapture(c, cudaStreamCaptureModeThreadLocal);
+  if (e != cudaSuccess) return e;
+  const cudaError_t ei = issue(c);
+  cudaGraph_t graph = nullptr;
+  e = cudaStreamEndCapture(c, &graph);
+  if (ei != cudaSuccess || e != cudaSuccess) {
+    if (graph) cudaGraphDestroy(graph);
+    cudaGetLastError();
+    return issue(st);   // (not capturable: issued directly)
+  }
+  cudaGraphExec_t exec = nullptr;
+  e = cudaGraphInstantiate(&exec, graph, 0);
+  cudaGraphDestroy(graph);
+  if (e != cudaSuccess) {
+    cudaGetLastError();
+    return issue(st);
+  }
+  if (cache.size() >= 16) {
+    for (Ent &x : cache) cudaGraphExecDestroy(x.exec);
+    cache.clear();
+  }
+  cache.push_back({key, exec});
+  return cudaGraphLaunch(exec, st);
+}
+
 static jp_status run_mode(const jp_loop *L, const Job &j, int mode, const jp_profile *prof, const jp_sched_cfg &c,
                           void *ws, size_t ws_bytes, jp_sched_result *res, cudaStream_t st, bool guide_ready = false,
                           int s_clean = 0, const int64_t *dist = nullptr) {
@@ -2218,8 +2262,24 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
     auto *bits = reinterpret_cast<uint32_t *>(pred + ((L->n + 63) & ~(int64_t)63));
     auto *V = at<unsigned long long>(ws, lg, R_TLS_C_A);
     const uint32_t *graw = at<uint32_t>(ws, lg, R_GUIDE);
-    JP_CUDA(launch_prof_pred(j, ws, lg, pred, bits, V, st), "last writers");   // (clears V[pred])
-    JP_CUDA(launch_tls_flow_waw(j, graw, pred, bits, V, &hd[H_TLS_COMMITTED], hd, st), "tls one window (waw)");
+    // the last-writer pass and the one-window kernel (five launches) replayed from
+    // a CUDA graph per loop / workspace: the host has just synchronised on the
+    // header, so every launch gap would be an idle GPU
+    auto issue9 = [&](cudaStream_t s) -> cudaError_t {
+      cudaError_t e = launch_prof_pred(j, ws, lg, pred, bits, V, s);   // (clears V[pred])
+      if (e == cudaSuccess) e = launch_tls_flow_waw(j, graw, pred, bits, V, &hd[H_TLS_COMMITTED], hd, s);
+      return e;
+    };
+    {
+      std::string key;
+      auto put = [&](auto v) { key.append(reinterpret_cast<const char *>(&v), sizeof v); };
+      int dev = 0;
+      cudaGetDevice(&dev);
+      put(dev); put(j.op); put(j.dt); put(j.d.n); put(j.d.ioff); put(j.d.base); put(j.d.lenA); put(j.d.r); put(j.d.w);
+      put(j.d.A); put(j.d.X); put(j.d.c0); put(ws); put(lg.total);
+      JP_CUDA(graph_launch(key, issue9, st), "last writers / tls one window (waw)");
+      note_launch(5);
+    }
     int64_t h2[H_PRED_SEG + 1];
     JP_CUDA(d2h_small_sync(h2, hd, sizeof h2, st), "tls D2H");
     if (h2[H_PRED_FAIL] == 0) {
