@@ -224,3 +224,33 @@ def test_large_A_profile_choice(la_log):
     wl = synth.Workload("largeA", O.OP_ADD_C, O.I32, n, A, r=torch.from_numpy(r), w=torch.from_numpy(w), c0=9)
     res = run_and_check(wl, expect_path=None)
     assert res["mode"] == jp.JP_MODE_TLS, res
+
+
+def test_graph_cache_alternating_loops():
+    """The profile (and path 9) replay CUDA graphs cached per argument set:
+    alternating two loops of the same shape on one workspace, and the same loop
+    after its index arrays changed in place (same pointers, new values), must
+    give the oracle's bytes every time."""
+    n = 1 << 20
+    a = synth.config3_waw(0.02, n=n, delta=1024)
+    b = synth.config3(0.02, n=n)
+    ga, gb = a.to(DEV), b.to(DEV)
+    La, Lb = jp.Loop.from_workload(ga), jp.Loop.from_workload(gb)
+    ws = jp.workspace(La)
+    ea, eb = to_oracle(a), to_oracle(b)
+    for rep in range(3):
+        for g, L, ref, path in ((ga, La, ea, 9), (gb, Lb, eb, 8)):
+            _, A, _ = O.run_seq(ref)
+            res = jp.jp_schedule(L, ws)
+            torch.cuda.synchronize()
+            assert res["tls_path"] == path and equal_bytes(g.A, A), (rep, res)
+            ref.A[:] = A
+    # new index values behind the same pointers (the graph replays the new data)
+    c = synth.config3_waw(0.05, n=n, delta=64)
+    ga.r.copy_(c.r.to(DEV))
+    ga.w.copy_(c.w.to(DEV))
+    ref = O.Loop(ea.op, ea.dtype, n, ga.A.cpu().numpy().copy(), r=c.r.numpy(), w=c.w.numpy(), c0=ea.c0)
+    _, A, _ = O.run_seq(ref)
+    res = jp.jp_schedule(La, ws)
+    torch.cuda.synchronize()
+    assert equal_bytes(ga.A, A), res
