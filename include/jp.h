@@ -462,13 +462,17 @@ jp_status jp_plan_tasks(const jp_loop *L, const int64_t *chunk_counts /* host */
                         void *ws, size_t ws_bytes, int64_t *tasks /* host [192] */, int32_t *n_tasks /* host */,
                         uint64_t *conf /* host [64] */, jp_stream_t st);
 /* jp_profile_plan_tasks: the same plan from a profile of the WHOLE loop L that
- * this call runs itself (every rank holds a full replica: no exchange, identical
+ * this call runs itself (the dependency-density profile of P:L191-196 with
+ * per-chunk counts, reading A19; the tasks and PDG of P:L197-200 / P:L441-442,
+ * reading B2; every rank holds a full replica: no exchange, identical
  * on every rank) -- by address buckets when L allows it (A >= 2^20, ADD_C /
  * SAXPY; then the task PDG first compares the per-chunk address ranges that
  * profile records), else stamp + classify.  prof (host): the loop's profile;
  * chunk_counts (host [3 * ceil(n / chunk_iters)]): per-chunk raw, war, waw;
- * tasks / n_tasks / conf as jp_plan_tasks.  JP_ERR_INDEX on an out-of-range
- * index (nothing modified).  syncs.                                          */
+ * tasks / n_tasks / conf as jp_plan_tasks.  ws: a workspace of L sized for
+ * JP_WS_ALL; its profile, key and scheduler regions are scratch of this call
+ * (JP_ERR_WORKSPACE when too small).  JP_ERR_INDEX on an out-of-range index
+ * (the loop's arrays are not modified).  syncs.                             */
 jp_status jp_profile_plan_tasks(const jp_loop *L, int64_t chunk_iters, double tau_high, void *ws, size_t ws_bytes,
                                 jp_profile *prof /* host */, int64_t *chunk_counts /* host */,
                                 int64_t *tasks /* host [192] */, int32_t *n_tasks /* host */,
