@@ -2204,7 +2204,12 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
         const uint32_t *g = at<uint32_t>(ws, lg, R_GUIDE);
         e = launch_tls_flow(j, g, g + (L->n + 31) / 32, at<unsigned long long>(ws, lg, R_TLS_C_A),
                             &hd[H_TLS_COMMITTED], st, nullptr, 0, hd, raw_max_for(L->n, c.tau_high),
-                            !bucket);   // (the bucket profile's reset of the header zeroed the statistics)
+                            !bucket,   // (the bucket profile's reset of the header zeroed the statistics)
+                            0,
+                            // the gather phase's values in region 1 (the bucket profile's records,
+                            // dead once its eval ran) for loops with few violators
+                            bucket && lg.bytes[R_MINW_A] >= 4 * (size_t)L->n ? at<uint32_t>(ws, lg, R_MINW_A) : nullptr,
+                            L->n / 64);
       }
       if (e == cudaSuccess) e = cudaEventSynchronize(ec);
       cudaEventDestroy(ep);

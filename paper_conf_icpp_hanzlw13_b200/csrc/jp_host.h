@@ -83,7 +83,10 @@ bool bucket_profile_ok(const Job &j, void *ws, const Layout &lo);
 cudaError_t launch_tls_flow(const Job &j, const uint32_t *graw, const uint32_t *gsrc, unsigned long long *V,
                             int64_t *stats, cudaStream_t st, const int32_t *wsrc = nullptr, int64_t lo = 0,
                             const int64_t *gate = nullptr, int64_t raw_max = 0, bool zero_stats = true,
-                            int max_ctas = 0);
+                            int max_ctas = 0, uint32_t *o = nullptr, int64_t ph_max = 0);
+// (o, n words of scratch, with a gate: when the gate's raw count is at most ph_max
+// the non-violators' values are gathered by a kernel of their own first and the
+// sweep only scatters them -- JP_FLOW_PHASED=0 keeps the one-kernel form)
 // wsrc (nullable, ADD_C): the first writer of every raw iteration's read (int32 [n])
 // crange (nullable, needs chunk % 16384 == 0): per chunk the min and max address of A
 // the chunk touches (uint32 [2 * chunks]) -- the stealing scheduler's task ranges

@@ -62,6 +62,8 @@ template <int DT>
 struct Flow {
   DLoop L;
   const uint32_t *graw, *gsrc;
+  const uint32_t *o;     // ph: every non-violator's value, from k_flow_gath
+  bool ph = false;
   unsigned long long *V;
   const int32_t *wsrc;   // nullable: writer of each raw iteration's read (loop-local id)
   uint32_t G, g, n, io, lo;
@@ -81,10 +83,15 @@ struct Flow {
     for (int k = 0; k < kFlowK; k++) {
       if (!act(base, k)) continue;
       const uint32_t i = it(base, k);
-      s.r[k] = L.r ? __ldcs(L.r + i) : (int32_t)(io + i);
       s.w[k] = L.w ? __ldcs(L.w + i) : (int32_t)(io + i);
       s.gr[k] = __ldcs(graw + (i >> 5));
       s.gs[k] = __ldcs(gsrc + (i >> 5));
+      if (ph) {   // the violators' read addresses; the others' values, gathered already
+        if (raw_bit(s, base, k)) s.r[k] = L.r ? __ldcs(L.r + i) : (int32_t)(io + i);
+        else s.x[k] = __ldcs(o + i);
+      } else {
+        s.r[k] = L.r ? __ldcs(L.r + i) : (int32_t)(io + i);
+      }
     }
     if (wsrc) {   // a range of a loop: a raw read written before the range reads A
 #pragma unroll
@@ -95,6 +102,7 @@ struct Flow {
   }
   // exposed reads of the non-violators (the violators' operands come from V)
   __device__ __forceinline__ void gather(uint32_t base, FlowSet &s) const {
+    if (ph) return;
 #pragma unroll
     for (int k = 0; k < kFlowK; k++)
       if (act(base, k) && !raw_bit(s, base, k)) s.x[k] = __ldcg(L.A + s.r[k]);
@@ -110,7 +118,7 @@ struct Flow {
     for (int k = 0; k < kFlowK; k++) {
       if (!act(base, k)) continue;
       if (raw_bit(s, base, k)) pend |= 1u << k;
-      else commit(s, base, k, op_add<DT>(s.x[k], L.c0));
+      else commit(s, base, k, ph ? s.x[k] : op_add<DT>(s.x[k], L.c0));
     }
     viol += __popc(pend);
     long long spins = 0;
@@ -137,7 +145,8 @@ struct Flow {
 template <int DT>
 __global__ void __launch_bounds__(kFlowT, JP_FLOW_MINB) k_tls_flow(DLoop L, const uint32_t *graw, const uint32_t *gsrc,
                                                        unsigned long long *V, int64_t *stats, const int32_t *wsrc,
-                                                       uint32_t lo, const int64_t *gate, int64_t raw_max) {
+                                                       uint32_t lo, const int64_t *gate, int64_t raw_max,
+                                                       const uint32_t *o, int64_t ph_max) {
   // gate (nullable): the profile header of this call -- launched before the host
   // has read it, the kernel runs only if the profile makes the loop a path-8 loop
   // (no bad index, war = waw = 0, 0 < raw <= raw_max, i.e. Fig. 2(b) mode B)
@@ -146,6 +155,9 @@ __global__ void __launch_bounds__(kFlowT, JP_FLOW_MINB) k_tls_flow(DLoop L, cons
     return;
   Flow<DT> F;
   F.L = L; F.graw = graw; F.gsrc = gsrc; F.V = V; F.wsrc = wsrc; F.lo = lo;
+  F.o = o;
+  // the gather kernel ran ahead (k_flow_gath) exactly when the gate's raw count is at most ph_max
+  F.ph = o && gate && gate[H_RAW] <= ph_max;
   F.G = gridDim.x * (uint32_t)kFlowT;
   F.g = blockIdx.x * (uint32_t)kFlowT + threadIdx.x;
   F.n = (uint32_t)L.n;
@@ -172,10 +184,53 @@ __global__ void __launch_bounds__(kFlowT, JP_FLOW_MINB) k_tls_flow(DLoop L, cons
   }
 }
 
+// The gather kernel of the phased sweep: o[i] = A[r[i]] + c0 for every
+// non-violator (its operand is never written, B12), gated like the sweep on the
+// profile header, plus raw <= ph_max.  2048 threads per SM (the sweep's register
+// budget allows 1024): the gathers at the device's random-read rate.
+template <int DT>
+__global__ void __launch_bounds__(256) k_flow_gath(DLoop L, const uint32_t *graw, uint32_t *o, const int64_t *gate,
+                                                   int64_t raw_max, int64_t ph_max) {
+  if (gate[H_BAD] != 0 || gate[H_WAR] != 0 || gate[H_WAW] != 0 || gate[H_RAW] <= 0 || gate[H_RAW] > raw_max ||
+      gate[H_GATE] != 0 || gate[H_RAW] > ph_max)
+    return;
+  constexpr int Q = 4;
+  const int64_t G = (int64_t)gridDim.x * blockDim.x;
+  for (int64_t i0 = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i0 < L.n; i0 += G * Q) {
+    int32_t r[Q];
+    uint32_t raw[Q], x[Q];
+#pragma unroll
+    for (int u = 0; u < Q; u++) {
+      const int64_t i = i0 + u * G;
+      raw[u] = 1;
+      if (i >= L.n) continue;
+      raw[u] = (__ldcs(graw + (i >> 5)) >> (i & 31)) & 1u;
+      r[u] = L.r ? __ldcs(L.r + i) : (int32_t)(L.ioff + i);
+    }
+#pragma unroll
+    for (int u = 0; u < Q; u++)
+      if (!raw[u]) x[u] = __ldcg(L.A + r[u]);
+#pragma unroll
+    for (int u = 0; u < Q; u++)
+      if (!raw[u]) __stcs(o + i0 + u * G, op_add<DT>(x[u], L.c0));
+  }
+}
+
+template <int DT>
+static cudaError_t run_flow_gath(const Job &j, const uint32_t *graw, uint32_t *o, const int64_t *gate, int64_t raw_max,
+                                 int64_t ph_max, cudaStream_t st) {
+  int64_t cap = (int64_t)num_sms() * 8;
+  const int64_t need = (j.d.n + 255) / 256;
+  const int grid = (int)(need < 1 ? 1 : need < cap ? need : cap);
+  k_flow_gath<DT><<<grid, 256, 0, st>>>(j.d, graw, o, gate, raw_max, ph_max);
+  note_launch();
+  return cudaSuccess;
+}
+
 template <int DT>
 static cudaError_t run_flow(const Job &j, const uint32_t *graw, const uint32_t *gsrc, unsigned long long *V,
                             int64_t *stats, cudaStream_t st, const int32_t *wsrc, uint32_t lo, const int64_t *gate,
-                            int64_t raw_max, int max_ctas) {
+                            int64_t raw_max, int max_ctas, const uint32_t *o, int64_t ph_max) {
   static int maxb = 0;   // (one device model per process: B200)
   if (maxb < 1) cudaOccupancyMaxActiveBlocksPerMultiprocessor(&maxb, (const void *)k_tls_flow<DT>, kFlowT, 0);
   if (maxb < 1) return cudaErrorInvalidConfiguration;
@@ -184,7 +239,7 @@ static cudaError_t run_flow(const Job &j, const uint32_t *graw, const uint32_t *
   const int64_t need = (j.d.n + kFlowT - 1) / kFlowT;
   if (need < grid) grid = (int)(need < 1 ? 1 : need);
   DLoop d = j.d;
-  void *args[] = {&d, &graw, &gsrc, &V, &stats, &wsrc, &lo, &gate, &raw_max};
+  void *args[] = {&d, &graw, &gsrc, &V, &stats, &wsrc, &lo, &gate, &raw_max, &o, &ph_max};
   note_launch();
   return cudaLaunchCooperativeKernel((const void *)k_tls_flow<DT>, dim3(grid), dim3(kFlowT), args, 0, st);
 }
@@ -376,12 +431,22 @@ cudaError_t launch_tls_flow_waw(const Job &j, const uint32_t *graw, const int32_
 // tagged 1 << 32 for an address the loop writes (zeroed).
 cudaError_t launch_tls_flow(const Job &j, const uint32_t *graw, const uint32_t *gsrc, unsigned long long *V,
                             int64_t *stats, cudaStream_t st, const int32_t *wsrc, int64_t lo, const int64_t *gate,
-                            int64_t raw_max, bool zero_stats, int max_ctas) {
+                            int64_t raw_max, bool zero_stats, int max_ctas, uint32_t *o, int64_t ph_max) {
   if (zero_stats) cudaMemsetAsync(stats, 0, 4 * sizeof(int64_t), st);
   if (j.d.n == 0) return launch_check();
   if (j.op != JP_OP_ADD_C) return cudaErrorInvalidValue;
-  cudaError_t e = j.dt == JP_F32 ? run_flow<JP_F32>(j, graw, gsrc, V, stats, st, wsrc, (uint32_t)lo, gate, raw_max, max_ctas)
-                                 : run_flow<JP_I32>(j, graw, gsrc, V, stats, st, wsrc, (uint32_t)lo, gate, raw_max, max_ctas);
+  // o with a gate: the non-violators' values gathered by a kernel of their own
+  // first (all the loop's random reads ahead of its writes: B200's L2 serves them
+  // faster apart, scripts/ubench/rand_phase.cu), when the gate's raw count is at
+  // most ph_max (few violators: the sweep then hardly waits)
+  const char *pe = getenv("JP_FLOW_PHASED");
+  if (!gate || (pe && pe[0] == '0')) o = nullptr;
+  cudaError_t e = cudaSuccess;
+  if (o) e = j.dt == JP_F32 ? run_flow_gath<JP_F32>(j, graw, o, gate, raw_max, ph_max, st)
+                            : run_flow_gath<JP_I32>(j, graw, o, gate, raw_max, ph_max, st);
+  if (e != cudaSuccess) return e;
+  e = j.dt == JP_F32 ? run_flow<JP_F32>(j, graw, gsrc, V, stats, st, wsrc, (uint32_t)lo, gate, raw_max, max_ctas, o, ph_max)
+                     : run_flow<JP_I32>(j, graw, gsrc, V, stats, st, wsrc, (uint32_t)lo, gate, raw_max, max_ctas, o, ph_max);
   if (e != cudaSuccess) return e;
   return launch_check();
 }
