@@ -1228,6 +1228,17 @@ static cudaError_t graph_launch(const std::string &key, const std::function<cuda
   return cudaGraphLaunch(exec, st);
 }
 
+// path 8's separate gather kernel runs up to this many raw iterations (a
+// fraction of n: 1/64 measured; JP_FLOW_PH_DIV overrides the divisor)
+static int64_t ph_max_for(int64_t n) {
+  static int64_t div = 0;
+  if (!div) {
+    const char *e = getenv("JP_FLOW_PH_DIV");
+    div = e ? std::max<int64_t>(1, atoll(e)) : 64;
+  }
+  return n / div;
+}
+
 static jp_status run_mode(const jp_loop *L, const Job &j, int mode, const jp_profile *prof, const jp_sched_cfg &c,
                           void *ws, size_t ws_bytes, jp_sched_result *res, cudaStream_t st, bool guide_ready = false,
                           int s_clean = 0, const int64_t *dist = nullptr) {
@@ -2209,7 +2220,7 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
                             // the gather phase's values in region 1 (the bucket profile's records,
                             // dead once its eval ran) for loops with few violators
                             bucket && lg.bytes[R_MINW_A] >= 4 * (size_t)L->n ? at<uint32_t>(ws, lg, R_MINW_A) : nullptr,
-                            L->n / 64);
+                            ph_max_for(L->n));
       }
       if (e == cudaSuccess) e = cudaEventSynchronize(ec);
       cudaEventDestroy(ep);
