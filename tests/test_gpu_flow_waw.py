@@ -254,3 +254,24 @@ def test_graph_cache_alternating_loops():
     res = jp.jp_schedule(La, ws)
     torch.cuda.synchronize()
     assert equal_bytes(ga.A, A), res
+
+
+@pytest.mark.parametrize("n", [1, 5, 1000, 16384, 16385, 40000])
+@pytest.mark.parametrize("kind", ["write_once", "waw"])
+def test_small_n_large_A(n, kind):
+    """Few iterations over a large A (the address-bucket profile with one or two
+    tiles, a partial last quad, most buckets empty): same bytes as the oracle."""
+    la = 1 << 20
+    g = np.random.default_rng(n + (7 if kind == "waw" else 0))
+    if kind == "write_once":
+        w = g.choice(la, size=n, replace=False).astype(np.int32)
+    else:
+        w = g.integers(0, max(2, n // 2), n).astype(np.int32)
+    r = w.copy()
+    dep = g.random(n) < 0.2
+    src = np.maximum(np.arange(n) - 1 - g.integers(0, 50, n), 0)
+    r[dep] = w[src[dep]]
+    r[0] = w[0]
+    A = torch.from_numpy(g.integers(-2**31, 2**31, size=la, dtype=np.int64).astype(np.int32))
+    wl = synth.Workload("small_n", O.OP_ADD_C, O.I32, n, A, r=torch.from_numpy(r), w=torch.from_numpy(w), c0=11)
+    run_and_check(wl, expect_path=None)
