@@ -298,6 +298,7 @@ __global__ void __launch_bounds__(kPh2Threads, 1) k_priv_tmp_2ph(DLoop L, unsign
   if (tid == 0)
     for (int64_t k = 0; k < kPh && k < my; k++) issue1(k);
   unsigned bad = 0;
+  bool full = false;   // this CTA's slot table has a writer in every slot
   for (int64_t k = 0; k < my; k++) {
     mbar_wait(&full1[k % kPh], (uint32_t)((k / kPh) & 1));
     const int64_t e0 = tile_of(k) * kPh2Tile;
@@ -314,18 +315,32 @@ __global__ void __launch_bounds__(kPh2Threads, 1) k_priv_tmp_2ph(DLoop L, unsign
       const int4 sv = S4[kPh2Tile / 4 - 1 - (q * kPh2Threads + tid)];   // descending in the tile
       sl[4 * q + 0] = sv.w; sl[4 * q + 1] = sv.z; sl[4 * q + 2] = sv.y; sl[4 * q + 3] = sv.x;
     }
+    if (full) {
+      // every slot already has a writer from a later tile of this CTA (tiles are
+      // walked in descending order): this tile only needs the index check
 #pragma unroll
-    for (int m = 0; m < 4 * kQ; m++) {
-      const bool ok = (uint32_t)sl[m] < lenT;
-      bad += !ok;
-      cur[m] = ok ? tT[sl[m]] : 0xFFFFFFFFu;
-    }
+      for (int m = 0; m < 4 * kQ; m++) bad += (uint32_t)sl[m] >= lenT;
+    } else {
 #pragma unroll
-    for (int m = 0; m < 4 * kQ; m++) {
-      const int q = m >> 2;
-      const int64_t i = e0 + 4 * (kPh2Tile / 4 - 1 - (q * kPh2Threads + tid)) + (3 - (m & 3));
-      const uint32_t v = (uint32_t)(i + 1);
-      if (cur[m] < v) atomicMax(&tT[sl[m]], v);
+      for (int m = 0; m < 4 * kQ; m++) {
+        const bool ok = (uint32_t)sl[m] < lenT;
+        bad += !ok;
+        cur[m] = ok ? tT[sl[m]] : 0xFFFFFFFFu;
+      }
+#pragma unroll
+      for (int m = 0; m < 4 * kQ; m++) {
+        const int q = m >> 2;
+        const int64_t i = e0 + 4 * (kPh2Tile / 4 - 1 - (q * kPh2Threads + tid)) + (3 - (m & 3));
+        const uint32_t v = (uint32_t)(i + 1);
+        if (cur[m] < v) atomicMax(&tT[sl[m]], v);
+      }
+      __syncthreads();
+      // a slot table this CTA has filled stays filled: later (lower) tiles of the
+      // CTA cannot hold a last writer (the coupon collector: 1024 slots are all
+      // seen within a tile or two of config 4's random s)
+      bool mine = true;
+      for (int64_t b = tid; b < (int64_t)lenT; b += kPh2Threads) mine = mine && tT[b] != 0;
+      full = __syncthreads_count(mine) == kPh2Threads;
     }
     __syncthreads();   // the stage is read: refill it
     if (tid == 0 && k + kPh < my) issue1(k + kPh);
