@@ -1968,8 +1968,9 @@ jp_status jp_schedule(const jp_loop *L, const jp_sched_cfg *cfgp, void *ws, size
             return fail(JP_ERR_CUDA, "tiny kernel finished without publishing its results");
         }
       }
-      JP_CUDA(cudaStreamSynchronize(st), "tiny sync");   // the kernel's tail: already done
-      memcpy(h, m.host, sizeof h);
+      // (no stream sync: the kernel publishes after its last write of A / T, and the
+      // arrays are read after st like every jp_schedule result, include/jp.h)
+      memcpy(h, const_cast<const int64_t *>(m.host), sizeof h);
     } else {
       JP_CUDA(launch_tiny(j, L, c.tau_high, c.tls_window, c.tls_w_max, c.tls_recovery, hdr, st), "tiny");
       JP_CUDA(d2h_small_sync(h, hdr, sizeof h, st), "tiny D2H");
