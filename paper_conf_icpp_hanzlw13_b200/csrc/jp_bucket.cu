@@ -163,14 +163,15 @@ __global__ void __launch_bounds__(kBThreads, 2) k_bk_count(BkView V, int vec, ui
 // the bucket total.  A bucket no iteration writes drops its pure reads (a read
 // with no writer of its address is neither raw nor the first read of a written
 // address: it changes no count, guide bit or table of the profile): wflag[b].
-// Block = 32 buckets (one per lane) x 32 tile segments (one per warp).
+// Block = 16 buckets x 64 tile segments (two segments per warp).
+constexpr int kScanNB = 16, kScanNS = 1024 / kScanNB;   // buckets x tile segments per CTA (B / 16 CTAs)
 __global__ void __launch_bounds__(1024) k_bk_scan_tiles(uint32_t *cnt, int T, int B, uint32_t *tot,
                                                          uint32_t *wflag, const int64_t *gate) {
   if (gated(gate)) return;
-  __shared__ uint32_t part_w[32][33], part_r[32][33];
-  const int lane = threadIdx.x & 31, seg = threadIdx.x >> 5;
-  const int b = blockIdx.x * 32 + lane;
-  const int per = (T + 31) / 32, t0 = seg * per, t1 = min(T, t0 + per);
+  __shared__ uint32_t part_w[kScanNS][kScanNB + 1], part_r[kScanNS][kScanNB + 1];
+  const int lane = threadIdx.x % kScanNB, seg = threadIdx.x / kScanNB;
+  const int b = blockIdx.x * kScanNB + lane;
+  const int per = (T + kScanNS - 1) / kScanNS, t0 = seg * per, t1 = min(T, t0 + per);
   uint32_t sw = 0, sr = 0;
   if (b < B)
 #pragma unroll 8
@@ -183,7 +184,7 @@ __global__ void __launch_bounds__(1024) k_bk_scan_tiles(uint32_t *cnt, int T, in
   part_r[seg][lane] = sr;
   __syncthreads();
   uint32_t allw = 0;
-  for (int k = 0; k < 32; k++) allw += part_w[k][lane];
+  for (int k = 0; k < kScanNS; k++) allw += part_w[k][lane];
   const bool keep = allw > 0;
   uint32_t run = 0;
   for (int k = 0; k < seg; k++) run += part_w[k][lane] + (keep ? part_r[k][lane] : 0u);
@@ -194,7 +195,7 @@ __global__ void __launch_bounds__(1024) k_bk_scan_tiles(uint32_t *cnt, int T, in
       cnt[(size_t)t * B + b] = run;
       run += (c & 0xFFFFu) + (keep ? c >> 16 : 0u);
     }
-    if (seg == 31) {
+    if (seg == kScanNS - 1) {
       tot[b] = run;
       wflag[b] = keep ? 1u : 0u;
     }
@@ -740,7 +741,7 @@ void run_bucket(const BkPlan &P, const DLoop &d, int64_t *hdr, BkOut O, cudaStre
   const int vec = al(d.r) && al(d.w);
   const int B = P.v.B, T = P.v.T;
   k_bk_count<OP><<<T, kBThreads, 4 * (size_t)B, st>>>(P.v, vec, P.cnt, &hdr[H_BAD]);
-  k_bk_scan_tiles<<<(B + 31) / 32, 1024, 0, st>>>(P.cnt, T, B, P.tot, P.wflag, P.v.gate);
+  k_bk_scan_tiles<<<(B + kScanNB - 1) / kScanNB, 1024, 0, st>>>(P.cnt, T, B, P.tot, P.wflag, P.v.gate);
   k_bk_scan_buckets<<<1, 1024, 0, st>>>(P.tot, B, P.base, P.order, P.v.gate);
   const size_t ssm = 6 * 2 * (size_t)kTile + 4 * (3 * (size_t)B + 1) + (size_t)B;
   k_bk_scatter<OP><<<T, kBThreads, ssm, st>>>(P.v, vec, P.cnt, P.tot, P.base, P.wflag, P.rec);
